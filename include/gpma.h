@@ -1,0 +1,169 @@
+/*
+ * gpma.h -- C ABI of the B200-native GPMA+ dynamic-graph store.
+ *
+ * The method is GPMA+ of Sha, Li, He, Tan, "Accelerating Dynamic Graph Analytics on
+ * GPUs", PVLDB 11(1), 2017 (cited as P:<line> of /root/reference/PAPER.md; R<n> are
+ * the readings listed in DESIGN.md / SURVEY.md §8(c)).
+ *
+ * Store: a packed memory array (PMA, §4.1) of edge keys (src<<32 | dst) with
+ * a u32 value, split into leaf segments of L slots; one guard entry (u, 0xFFFFFFFF)
+ * per vertex u marks the end of row u so that row_offset[u+1] = slot(guard u) turns
+ * the gapped array into a CSR (CSR on GPMA, §4.2, Fig. 5).
+ *
+ * Conventions for every entry point
+ *   - Pointers to arrays may be DEVICE pointers (cudaMalloc / torch CUDA tensors) or
+ *     HOST pointers (pinned or pageable); the library detects the kind with
+ *     cudaPointerGetAttributes and stages host buffers through its own device memory
+ *     on the given stream.  The library never retains a caller pointer past the call.
+ *   - Calls are stream-ordered on `stream` (NULL = legacy default stream).  With device
+ *     outputs the caller may read them after synchronising the stream; with host
+ *     outputs the call synchronises the stream before returning.
+ *   - The library owns all store memory (cudaMallocAsync on the call's stream).
+ *   - Every function returns a gpma_status.  Argument, range and reserved-value
+ *     errors are detected before anything is mutated (no partial batch).  A CUDA
+ *     error poisons the handle; later calls return GPMA_ERR_POISONED.
+ *   - A handle is not thread-safe; use it from one host thread / stream at a time.
+ *   - All compute runs in the sm_100a kernels of this library; there is no CPU path.
+ */
+#ifndef GPMA_H
+#define GPMA_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+struct CUstream_st;                       /* cudaStream_t == struct CUstream_st* */
+typedef struct CUstream_st *gpma_stream_t;
+typedef struct gpma gpma_t;               /* opaque: one store (or one shard)     */
+
+typedef enum {
+  GPMA_OK = 0,
+  GPMA_ERR_INVALID_ARG = 1, /* NULL handle/pointer, bad op, bad config             */
+  GPMA_ERR_RANGE = 2,       /* a src or dst >= num_vertices (R23)                   */
+  GPMA_ERR_RESERVED = 3,    /* dst == 0xFFFFFFFF (guard column, R1) or
+                               val == 0xFFFFFFFF (tombstone, R12)                   */
+  GPMA_ERR_OOM = 4,         /* device allocation failed                             */
+  GPMA_ERR_CUDA = 5,        /* a CUDA call failed; the handle is now poisoned       */
+  GPMA_ERR_POISONED = 6     /* an earlier CUDA error poisoned this handle           */
+} gpma_status;
+
+typedef enum { GPMA_INSERT = 0, GPMA_DELETE = 1 } gpma_op;
+
+/* R12: deletions are either lazy (the paper's sliding-window mode: mark
+ * the slot deleted, no density maintenance, recycled by later rewrites) or the dual of
+ * insertion (lower-bound test per level, root halving). */
+typedef enum { GPMA_DELETE_LAZY = 0, GPMA_DELETE_REBALANCE = 1 } gpma_delete_mode;
+
+typedef struct {
+  uint32_t struct_size;       /* sizeof(gpma_config)                                  */
+  uint32_t leaf_slots;        /* L; 0 = R3 rule max(4, 2^floor(log2 log2 cap0)).
+                                 Must be a power of two in [4, 32].                   */
+  uint64_t initial_capacity;  /* 0 = R15 rule (smallest 2^k >= 8 holding E0+V at
+                                 init_density_bp); else a power of two >= 2L          */
+  uint16_t rho_leaf_bp, rho_root_bp, tau_leaf_bp, tau_root_bp; /* R4, basis points:
+                                 800, 4000, 9200, 8000 = Fig. 3           */
+  uint16_t init_density_bp;   /* R15: 6000                                            */
+  uint16_t reserved0;
+  uint32_t delete_mode;       /* gpma_delete_mode                                     */
+} gpma_config;
+
+typedef struct {
+  uint32_t num_vertices;
+  uint32_t leaf_slots;        /* L                                                    */
+  uint64_t capacity;          /* slots (power of two)                                 */
+  uint32_t height;            /* h: capacity = L * 2^h                                */
+  uint32_t delete_mode;
+  uint64_t live_edges;        /* live entries excluding guards                        */
+  uint64_t tombstones;        /* lazily deleted entries still occupying slots         */
+  uint64_t resizes;           /* root doublings + halvings since create               */
+  /* last gpma_update_batch: */
+  uint64_t last_unique;       /* distinct keys in the batch                           */
+  uint64_t last_pending;      /* updates entering the level loop after the pre-pass   */
+  uint64_t last_slots_rewritten;   /* sum of |W| over re-dispatched windows (+ resize) */
+  uint64_t last_windows_rewritten;
+  uint32_t last_top_level;    /* highest level reached (h+1 = resized)                */
+  uint32_t last_resized;
+} gpma_stats_t;
+
+/* Fill *cfg with the defaults above. */
+void gpma_config_default(gpma_config *cfg);
+
+/* Build a store over vertices [0, num_vertices) from n_init edges (keys u64[n_init],
+ * vals u32[n_init]; may repeat, the last occurrence wins, R10).  Inserts the V guards
+ * (R1), picks capacity (R15) and leaf size (R3), lays everything out evenly (R7).
+ * cfg may be NULL (defaults).  On success *out owns the store. */
+gpma_status gpma_create(uint32_t num_vertices, const uint64_t *init_keys,
+                        const uint32_t *init_vals, uint64_t n_init, const gpma_config *cfg,
+                        gpma_stream_t stream, gpma_t **out);
+
+/* Test hook: load a raw slot layout keys u64[capacity], vals u32[capacity] (e.g. the
+ * Fig. 3 PMA) with leaf size leaf_slots; guards are optional.  The layout must
+ * be sorted over occupied slots and left-packed per leaf. */
+gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t leaf_slots,
+                            const uint64_t *keys, const uint32_t *vals, const gpma_config *cfg,
+                            gpma_stream_t stream, gpma_t **out);
+
+gpma_status gpma_destroy(gpma_t *g);
+
+/* Apply one homogeneous batch (Alg. 4): keys u64[n] (src<<32|dst), vals
+ * u32[n] (ignored and may be NULL for GPMA_DELETE).  Keys may be unsorted and repeat
+ * (last occurrence wins).  INSERT of a live key overwrites its value; of a tombstoned
+ * key revives it in place (R11, R12).  DELETE of an absent key is a no-op (R13).
+ * n == 0 is a no-op.  Errors: RANGE / RESERVED before any mutation. */
+gpma_status gpma_update_batch(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
+                              gpma_op op, gpma_stream_t stream);
+
+/* BFS from root over the live out-edges (Alg. 2-3):
+ * levels i32[V] = hop distance, -1 if unreachable. */
+gpma_status gpma_bfs(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t stream);
+
+/* Weakly connected components (R19): labels u32[V] = the minimum vertex
+ * id of each vertex's component. */
+gpma_status gpma_cc(gpma_t *g, uint32_t *labels, gpma_stream_t stream);
+
+/* PageRank by power iteration (R20/R21):
+ *   x'[v] = (1-d)/V + d * (sum_{u->v} x[u]/outdeg(u) + D/V),  D = sum of dangling x[u];
+ * stops after the first iteration with ||x'-x||_1 < tol_l1 (tol 0 = exactly max_iter
+ * iterations).  rank f64[V]: input when warm_start != 0, else
+ * initialised to 1/V; output = the last x'.  *iters_out (may be NULL) = iterations. */
+gpma_status gpma_pagerank(gpma_t *g, double *rank, int warm_start, double damping,
+                          double tol_l1, int max_iter, int *iters_out, gpma_stream_t stream);
+/* Same in fp32 (accumulation in fp32). */
+gpma_status gpma_pagerank_f32(gpma_t *g, float *rank, int warm_start, float damping,
+                              float tol_l1, int max_iter, int *iters_out, gpma_stream_t stream);
+
+/* CSR view (Fig. 5): row_ptr u64[V+1], col u32[nnz], val u32[nnz]
+ * of the live edges in key order.  col == NULL: only *nnz_out is computed (size
+ * query).  nnz_capacity < nnz -> GPMA_ERR_INVALID_ARG with *nnz_out set. */
+gpma_status gpma_export_csr(gpma_t *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
+                            uint64_t nnz_capacity, uint64_t *nnz_out, gpma_stream_t stream);
+
+gpma_status gpma_stats(gpma_t *g, gpma_stats_t *out);
+
+/* Parity hooks.  Raw layout: keys u64[capacity] (0xFFFF..FF = empty), vals
+ * u32[capacity] (0 on empty slots); row_offset u64[V+1] (R8); leaf_live u32[cap/L]
+ * (live entries incl. guards per leaf); heads u64[cap/L] (locate index, R9).  Any
+ * output pointer may be NULL. */
+gpma_status gpma_debug_dump(gpma_t *g, uint64_t *keys, uint32_t *vals, uint64_t *row_offset,
+                            uint32_t *leaf_live, uint64_t *heads, gpma_stream_t stream);
+
+/* Per-level trace of the following update batches (Fig. 6 "Update Segments /
+ * Offsets / Successful Flag"), off by default (it adds host syncs). */
+gpma_status gpma_debug_set_trace(gpma_t *g, int enable);
+/* Records (level, seg_start_slot, offset, flag) x4 u64; flag 2 closes a level and
+ * carries the final offset.  Returns the record count in *count; copies at most max. */
+gpma_status gpma_debug_trace(gpma_t *g, uint64_t *out4, uint64_t max, uint64_t *count);
+
+/* Number of kernels this handle has launched since create (bench evidence). */
+uint64_t gpma_kernel_launches(const gpma_t *g);
+
+const char *gpma_status_string(gpma_status s);
+const char *gpma_last_error(const gpma_t *g);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* GPMA_H */

@@ -1,0 +1,390 @@
+// capi.cu -- the extern "C" boundary declared in include/gpma.h.
+// Argument checking, host/device pointer staging and handle lifetime only; every step
+// of the method runs in the kernels of update.cu / analytics.cu / primitives.cu.
+#include <cuda_runtime.h>
+#include <string.h>
+
+#include <new>
+
+#include "gpma_internal.cuh"
+
+using gp::DevBuf;
+
+namespace {
+
+bool is_host_ptr(const void *p) {
+  if (!p) return false;
+  cudaPointerAttributes at;
+  if (cudaPointerGetAttributes(&at, p) != cudaSuccess) {
+    cudaGetLastError();
+    return true;
+  }
+  return !(at.type == cudaMemoryTypeDevice || at.type == cudaMemoryTypeManaged);
+}
+
+// Output staging: kernels always write device memory; a host destination is filled
+// by a D2H copy at the end of the call (which then synchronises the stream).
+struct Out {
+  gpma *g;
+  void *user;
+  size_t bytes;
+  bool host;
+  DevBuf buf;
+  cudaStream_t s;
+  Out(gpma *g_, void *u, size_t b, cudaStream_t s_) : g(g_), user(u), bytes(b), host(is_host_ptr(u)), s(s_) {}
+  ~Out() { gp::release(buf, s); }
+  cudaError_t dev(void **p, bool copy_in) {
+    if (!user) { *p = nullptr; return cudaSuccess; }
+    if (!host) { *p = user; return cudaSuccess; }
+    cudaError_t e = gp::ensure(buf, bytes, s);
+    if (e) return e;
+    if (copy_in) {
+      e = cudaMemcpyAsync(buf.p, user, bytes, cudaMemcpyHostToDevice, s);
+      if (e) return e;
+    }
+    *p = buf.p;
+    return cudaSuccess;
+  }
+  cudaError_t finish() {
+    if (!user || !host) return cudaSuccess;
+    cudaError_t e = cudaMemcpyAsync(user, buf.p, bytes, cudaMemcpyDeviceToHost, s);
+    if (e) return e;
+    return cudaStreamSynchronize(s);
+  }
+};
+
+gpma_status begin(gpma *g) {
+  if (!g) return GPMA_ERR_INVALID_ARG;
+  if (g->poisoned) return GPMA_ERR_POISONED;
+  g->err.clear();
+  return GPMA_OK;
+}
+
+gpma_status end(gpma *g, gpma_status st) {
+  if (st == GPMA_OK) {
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return gp::cuda_fail(g, e, "kernel launch");
+  }
+  return st;
+}
+
+gpma_status apply_config(gpma *g, const gpma_config *cfg, uint32_t *leaf, uint64_t *cap) {
+  gpma_config c;
+  gpma_config_default(&c);
+  if (cfg) {
+    if (cfg->struct_size < sizeof(uint32_t) * 2) return GPMA_ERR_INVALID_ARG;
+    size_t n = cfg->struct_size < sizeof(c) ? cfg->struct_size : sizeof(c);
+    memcpy(&c, cfg, n);
+  }
+  if (c.leaf_slots && (c.leaf_slots < 4 || c.leaf_slots > 32 || (c.leaf_slots & (c.leaf_slots - 1))))
+    return GPMA_ERR_INVALID_ARG;
+  if (c.delete_mode > 1) return GPMA_ERR_INVALID_ARG;
+  if (c.rho_leaf_bp > 10000 || c.rho_root_bp > 10000 || c.tau_leaf_bp > 10000 || c.tau_root_bp > 10000 ||
+      c.init_density_bp == 0 || c.init_density_bp > 10000)
+    return GPMA_ERR_INVALID_ARG;
+  g->rho0 = c.rho_leaf_bp;
+  g->rhoh = c.rho_root_bp;
+  g->tau0 = c.tau_leaf_bp;
+  g->tauh = c.tau_root_bp;
+  g->init_bp = c.init_density_bp;
+  g->mode = c.delete_mode;
+  *leaf = c.leaf_slots;
+  *cap = c.initial_capacity;
+  return GPMA_OK;
+}
+
+gpma *new_handle(uint32_t V) {
+  gpma *g = new (std::nothrow) gpma();
+  if (!g) return nullptr;
+  g->V = V;
+  if (cudaMalloc((void **)&g->ctrl_d, sizeof(gp::Ctrl)) != cudaSuccess ||
+      cudaMallocHost((void **)&g->ctrl_h, sizeof(gp::Ctrl)) != cudaSuccess) {
+    cudaGetLastError();
+    if (g->ctrl_d) cudaFree(g->ctrl_d);
+    delete g;
+    return nullptr;
+  }
+  memset(g->ctrl_h, 0, sizeof(gp::Ctrl));
+  return g;
+}
+
+void free_handle(gpma *g) {
+  if (!g) return;
+  cudaStream_t s = g->st;
+  DevBuf *bufs[] = {&g->b_sk[0], &g->b_sk[1], &g->b_sv[0], &g->b_sv[1], &g->b_keep, &g->b_pos, &g->b_tgt,
+                    &g->b_pk[0], &g->b_pk[1], &g->b_pv[0], &g->b_pv[1], &g->b_pt[0], &g->b_pt[1],
+                    &g->b_hf, &g->b_widx, &g->b_wfirst, &g->b_acc, &g->b_aidx, &g->b_alist, &g->b_nw,
+                    &g->b_woff, &g->b_keep2, &g->b_kpos, &g->b_lpre, &g->b_wk, &g->b_wv, &g->b_dirty,
+                    &g->b_scan, &g->b_hist, &g->b_stage[0], &g->b_stage[1], &g->b_stage[2],
+                    &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3};
+  for (DevBuf *b : bufs) gp::release(*b, s);
+  if (g->key) cudaFreeAsync(g->key, s);
+  if (g->val) cudaFreeAsync(g->val, s);
+  if (g->cnt) cudaFreeAsync(g->cnt, s);
+  if (g->head) cudaFreeAsync(g->head, s);
+  if (g->row_offset) cudaFreeAsync(g->row_offset, s);
+  cudaStreamSynchronize(s);
+  if (g->ctrl_d) cudaFree(g->ctrl_d);
+  if (g->ctrl_h) cudaFreeHost(g->ctrl_h);
+  cudaGetLastError();
+  delete g;
+}
+
+}  // namespace
+
+namespace gp {
+gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
+                              uint64_t cap_override, uint32_t leaf_override, cudaStream_t s);
+}
+
+extern "C" {
+
+void gpma_config_default(gpma_config *cfg) {
+  if (!cfg) return;
+  memset(cfg, 0, sizeof(*cfg));
+  cfg->struct_size = sizeof(gpma_config);
+  cfg->leaf_slots = 0;
+  cfg->initial_capacity = 0;
+  cfg->rho_leaf_bp = 800;
+  cfg->rho_root_bp = 4000;
+  cfg->tau_leaf_bp = 9200;
+  cfg->tau_root_bp = 8000;
+  cfg->init_density_bp = 6000;
+  cfg->delete_mode = GPMA_DELETE_LAZY;
+}
+
+gpma_status gpma_create(uint32_t num_vertices, const uint64_t *init_keys, const uint32_t *init_vals,
+                        uint64_t n_init, const gpma_config *cfg, gpma_stream_t stream, gpma_t **out) {
+  if (!out || num_vertices == 0 || num_vertices == 0xFFFFFFFFu) return GPMA_ERR_INVALID_ARG;
+  if (n_init && (!init_keys || !init_vals)) return GPMA_ERR_INVALID_ARG;
+  *out = nullptr;
+  gpma *g = new_handle(num_vertices);
+  if (!g) return GPMA_ERR_OOM;
+  cudaStream_t s = (cudaStream_t)stream;
+  g->st = s;
+  uint32_t leaf = 0;
+  uint64_t cap = 0;
+  gpma_status st = apply_config(g, cfg, &leaf, &cap);
+  if (st == GPMA_OK && cap && (cap & (cap - 1))) st = GPMA_ERR_INVALID_ARG;
+  if (st == GPMA_OK) st = gp::create_from_batch(g, init_keys, init_vals, n_init, cap, leaf, s);
+  if (st == GPMA_OK) {
+    cudaError_t e = cudaStreamSynchronize(s);
+    if (e) st = gp::cuda_fail(g, e, "create");
+  }
+  if (st != GPMA_OK) {
+    free_handle(g);
+    return st;
+  }
+  *out = g;
+  return GPMA_OK;
+}
+
+gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t leaf_slots,
+                            const uint64_t *keys, const uint32_t *vals, const gpma_config *cfg,
+                            gpma_stream_t stream, gpma_t **out) {
+  if (!out || !keys || !vals || num_vertices == 0) return GPMA_ERR_INVALID_ARG;
+  if (leaf_slots < 4 || leaf_slots > 32 || (leaf_slots & (leaf_slots - 1))) return GPMA_ERR_INVALID_ARG;
+  if (capacity < 2ull * leaf_slots || (capacity & (capacity - 1))) return GPMA_ERR_INVALID_ARG;
+  *out = nullptr;
+  gpma *g = new_handle(num_vertices);
+  if (!g) return GPMA_ERR_OOM;
+  cudaStream_t s = (cudaStream_t)stream;
+  g->st = s;
+  uint32_t leaf = 0;
+  uint64_t cap = 0;
+  gpma_status st = apply_config(g, cfg, &leaf, &cap);
+  if (st == GPMA_OK) {
+    g->L = leaf_slots;
+    g->cap = capacity;
+    g->h = gp::ilog2(capacity / leaf_slots);
+    gp::level_bounds(g->L, g->h, g->rho0, g->rhoh, g->tau0, g->tauh, g->tmin, g->tmax);
+    uint64_t nl = capacity / leaf_slots;
+    if (cudaMallocAsync((void **)&g->key, capacity * 8, s) || cudaMallocAsync((void **)&g->val, capacity * 4, s) ||
+        cudaMallocAsync((void **)&g->cnt, nl * 4, s) || cudaMallocAsync((void **)&g->head, nl * 8, s) ||
+        cudaMallocAsync((void **)&g->row_offset, ((uint64_t)num_vertices + 1) * 8, s)) {
+      cudaGetLastError();
+      st = GPMA_ERR_OOM;
+    }
+  }
+  if (st == GPMA_OK) {
+    cudaMemsetAsync(g->row_offset, 0, ((uint64_t)num_vertices + 1) * 8, s);
+    st = gp::load_raw(g, keys, vals, s);
+  }
+  if (st == GPMA_OK && cudaStreamSynchronize(s) != cudaSuccess) st = GPMA_ERR_CUDA;
+  if (st != GPMA_OK) {
+    free_handle(g);
+    return st;
+  }
+  *out = g;
+  return GPMA_OK;
+}
+
+gpma_status gpma_destroy(gpma_t *g) {
+  if (!g) return GPMA_ERR_INVALID_ARG;
+  free_handle(g);
+  return GPMA_OK;
+}
+
+gpma_status gpma_update_batch(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, gpma_op op,
+                              gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (op != GPMA_INSERT && op != GPMA_DELETE) return GPMA_ERR_INVALID_ARG;
+  if (n && !keys) return GPMA_ERR_INVALID_ARG;
+  if (n && op == GPMA_INSERT && !vals) return GPMA_ERR_INVALID_ARG;
+  if (n > 0xFFFFFFFFull) return GPMA_ERR_INVALID_ARG;
+  g->st = (cudaStream_t)stream;
+  return end(g, gp::update_batch(g, keys, vals, n, (int)op, (cudaStream_t)stream));
+}
+
+gpma_status gpma_bfs(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!levels || root >= g->V) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  Out o(g, levels, (size_t)g->V * 4, s);
+  void *d;
+  if (cudaError_t e = o.dev(&d, false)) return gp::cuda_fail(g, e, "bfs staging");
+  st = gp::bfs(g, root, (int32_t *)d, s);
+  if (st == GPMA_OK)
+    if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "bfs copy-out");
+  return end(g, st);
+}
+
+gpma_status gpma_cc(gpma_t *g, uint32_t *labels, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!labels) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  Out o(g, labels, (size_t)g->V * 4, s);
+  void *d;
+  if (cudaError_t e = o.dev(&d, false)) return gp::cuda_fail(g, e, "cc staging");
+  st = gp::cc(g, (uint32_t *)d, s);
+  if (st == GPMA_OK)
+    if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "cc copy-out");
+  return end(g, st);
+}
+
+gpma_status gpma_pagerank(gpma_t *g, double *rank, int warm_start, double damping, double tol_l1, int max_iter,
+                          int *iters_out, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!rank || max_iter < 0 || !(damping >= 0.0 && damping <= 1.0) || !(tol_l1 >= 0.0)) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  Out o(g, rank, (size_t)g->V * 8, s);
+  void *d;
+  if (cudaError_t e = o.dev(&d, warm_start != 0)) return gp::cuda_fail(g, e, "pagerank staging");
+  st = gp::pagerank_f64(g, (double *)d, warm_start, damping, tol_l1, max_iter, iters_out, s);
+  if (st == GPMA_OK)
+    if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "pagerank copy-out");
+  return end(g, st);
+}
+
+gpma_status gpma_pagerank_f32(gpma_t *g, float *rank, int warm_start, float damping, float tol_l1, int max_iter,
+                              int *iters_out, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!rank || max_iter < 0 || !(damping >= 0.0f && damping <= 1.0f) || !(tol_l1 >= 0.0f)) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  Out o(g, rank, (size_t)g->V * 4, s);
+  void *d;
+  if (cudaError_t e = o.dev(&d, warm_start != 0)) return gp::cuda_fail(g, e, "pagerank staging");
+  st = gp::pagerank_f32(g, (float *)d, warm_start, damping, tol_l1, max_iter, iters_out, s);
+  if (st == GPMA_OK)
+    if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "pagerank copy-out");
+  return end(g, st);
+}
+
+gpma_status gpma_export_csr(gpma_t *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val, uint64_t nnz_capacity,
+                            uint64_t *nnz_out, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (col && (!row_ptr || !val)) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  uint64_t nnz = 0;
+  if (!col) {
+    st = gp::export_csr(g, nullptr, nullptr, nullptr, 0, &nnz, s);
+    if (nnz_out) *nnz_out = nnz;
+    return end(g, st);
+  }
+  Out orp(g, row_ptr, ((size_t)g->V + 1) * 8, s), oc(g, col, (size_t)nnz_capacity * 4, s),
+      ov(g, val, (size_t)nnz_capacity * 4, s);
+  void *drp, *dc, *dv;
+  if (cudaError_t e = orp.dev(&drp, false)) return gp::cuda_fail(g, e, "export staging");
+  if (cudaError_t e = oc.dev(&dc, false)) return gp::cuda_fail(g, e, "export staging");
+  if (cudaError_t e = ov.dev(&dv, false)) return gp::cuda_fail(g, e, "export staging");
+  st = gp::export_csr(g, (uint64_t *)drp, (uint32_t *)dc, (uint32_t *)dv, nnz_capacity, &nnz, s);
+  if (nnz_out) *nnz_out = nnz;
+  if (st == GPMA_OK) {
+    oc.bytes = (size_t)nnz * 4;
+    ov.bytes = (size_t)nnz * 4;
+    cudaError_t e;
+    if ((e = orp.finish()) || (e = oc.finish()) || (e = ov.finish())) return gp::cuda_fail(g, e, "export copy-out");
+  }
+  return end(g, st);
+}
+
+gpma_status gpma_stats(gpma_t *g, gpma_stats_t *out) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!out) return GPMA_ERR_INVALID_ARG;
+  *out = g->last;
+  out->num_vertices = g->V;
+  out->leaf_slots = g->L;
+  out->capacity = g->cap;
+  out->height = g->h;
+  out->delete_mode = g->mode;
+  out->resizes = g->resizes;
+  st = gp::count_slots(g, &out->live_edges, &out->tombstones, g->st);
+  return end(g, st);
+}
+
+gpma_status gpma_debug_dump(gpma_t *g, uint64_t *keys, uint32_t *vals, uint64_t *row_offset, uint32_t *leaf_live,
+                            uint64_t *heads, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  cudaStream_t s = (cudaStream_t)stream;
+  uint64_t nl = g->cap / g->L;
+  struct { void *dst; const void *src; size_t bytes; } cp[] = {
+      {keys, g->key, g->cap * 8}, {vals, g->val, g->cap * 4}, {row_offset, g->row_offset, ((size_t)g->V + 1) * 8},
+      {leaf_live, g->cnt, nl * 4}, {heads, g->head, nl * 8}};
+  for (auto &c : cp)
+    if (c.dst)
+      if (cudaError_t e = cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDefault, s))
+        return gp::cuda_fail(g, e, "debug_dump");
+  if (cudaError_t e = cudaStreamSynchronize(s)) return gp::cuda_fail(g, e, "debug_dump");
+  return GPMA_OK;
+}
+
+gpma_status gpma_debug_set_trace(gpma_t *g, int enable) {
+  if (!g) return GPMA_ERR_INVALID_ARG;
+  g->trace_on = enable != 0;
+  return GPMA_OK;
+}
+
+gpma_status gpma_debug_trace(gpma_t *g, uint64_t *out4, uint64_t max, uint64_t *count) {
+  if (!g || !count) return GPMA_ERR_INVALID_ARG;
+  uint64_t n = g->trace.size() / 4;
+  *count = n;
+  if (out4) memcpy(out4, g->trace.data(), (n < max ? n : max) * 4 * sizeof(uint64_t));
+  return GPMA_OK;
+}
+
+uint64_t gpma_kernel_launches(const gpma_t *g) { return g ? g->launches : 0; }
+
+const char *gpma_status_string(gpma_status s) {
+  switch (s) {
+    case GPMA_OK: return "ok";
+    case GPMA_ERR_INVALID_ARG: return "invalid argument";
+    case GPMA_ERR_RANGE: return "vertex id out of range";
+    case GPMA_ERR_RESERVED: return "reserved key or value";
+    case GPMA_ERR_OOM: return "out of device memory";
+    case GPMA_ERR_CUDA: return "CUDA error";
+    case GPMA_ERR_POISONED: return "handle poisoned by an earlier CUDA error";
+  }
+  return "unknown";
+}
+
+const char *gpma_last_error(const gpma_t *g) { return g ? g->err.c_str() : "null handle"; }
+
+}  // extern "C"

@@ -1,0 +1,153 @@
+// gpma_internal.cuh -- internal definitions of the sm_100a GPMA+ library.
+// Paper: Sha et al., PVLDB 11(1) 2017 (PAPER.md, cited P:<line>); readings R<n> in DESIGN.md.
+#pragma once
+
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include <string>
+#include <vector>
+
+#include "../../include/gpma.h"
+
+namespace gp {
+
+constexpr uint64_t KEY_NONE = ~0ull;          // R2 empty slot
+constexpr uint32_t VAL_TOMB = 0xFFFFFFFFu;    // R12 lazy-delete mark
+constexpr uint32_t COL_GUARD = 0xFFFFFFFFu;   // R1 guard column ("infinity")
+constexpr int MAX_RESIDENT_BLOCKS = 148 * 8;  // grid-stride kernels: 8 x 256-thread CTAs per SM
+
+__host__ __device__ inline bool is_guard_key(uint64_t k) {
+  return k != KEY_NONE && (uint32_t)k == COL_GUARD;
+}
+
+struct DevBuf {
+  void *p = nullptr;
+  size_t bytes = 0;
+};
+
+// Device-side control block (counters written by kernels, read back in one copy).
+struct Ctrl {
+  uint32_t err;            // validation bits: 1 = range, 2 = reserved
+  uint32_t pad0;
+  uint64_t nunique;        // distinct keys in the batch
+  uint64_t slots_rewritten;
+  uint64_t windows_rewritten;
+  uint64_t ndirty;         // dirty windows recorded for the head fix-up
+  uint64_t sum;            // scratch reductions
+  uint64_t sum2;
+};
+
+// Per-level descriptors of one GPMA+ round (Alg. 4 l.7-15).
+struct LevelBufs {
+  uint32_t *hf = nullptr;     // [p+1] window-head flags -> exclusive scan (widx)
+  uint32_t *widx = nullptr;
+  uint32_t *wfirst = nullptr; // [p+1] offsets I
+  uint32_t *acc = nullptr;    // [p+1] success flags -> aidx
+  uint32_t *aidx = nullptr;
+  uint32_t *alist = nullptr;  // accepted window ids
+  uint64_t *nw = nullptr;     // [p+1] entries after merge -> woff
+  uint64_t *woff = nullptr;
+  uint32_t *keep = nullptr;   // [p+1]
+  uint32_t *kpos = nullptr;
+};
+
+}  // namespace gp
+
+struct gpma {
+  // geometry (R3, R4, R5, R15)
+  uint32_t V = 0, L = 0, h = 0, mode = 0;
+  uint64_t cap = 0;
+  uint32_t rho0 = 800, rhoh = 4000, tau0 = 9200, tauh = 8000, init_bp = 6000;
+  std::vector<uint64_t> tmin, tmax;
+
+  // store (HBM-resident)
+  uint64_t *key = nullptr;        // [cap]
+  uint32_t *val = nullptr;        // [cap]
+  uint32_t *cnt = nullptr;        // [cap/L] live entries (incl. guards) per leaf
+  uint64_t *head = nullptr;       // [cap/L] locate index (R9)
+  uint64_t *row_offset = nullptr; // [V+1] (R8)
+
+  // scratch arena
+  gp::DevBuf b_sk[2], b_sv[2], b_keep, b_pos, b_tgt;       // batch
+  gp::DevBuf b_pk[2], b_pv[2], b_pt[2];                      // pending (ping-pong)
+  gp::DevBuf b_hf, b_widx, b_wfirst, b_acc, b_aidx, b_alist, b_nw, b_woff, b_keep2, b_kpos;
+  gp::DevBuf b_lpre, b_wk, b_wv, b_dirty, b_scan, b_hist, b_stage[4], b_misc, b_misc2, b_misc3;
+  gp::Ctrl *ctrl_d = nullptr;
+  gp::Ctrl *ctrl_h = nullptr;     // pinned mirror
+
+  // state
+  bool poisoned = false;
+  std::string err;
+  uint64_t launches = 0;
+  uint64_t resizes = 0;
+  gpma_stats_t last{};
+  bool trace_on = false;
+  std::vector<uint64_t> trace;    // (level, start, offset, flag) x4
+  cudaStream_t st = nullptr;
+};
+
+// ---------------------------------------------------------------- helpers (host)
+namespace gp {
+
+#define GP_LAUNCH(g, kernel, grid, block, smem, stream, ...)                 \
+  do {                                                                       \
+    kernel<<<(grid), (block), (smem), (stream)>>>(__VA_ARGS__);              \
+    (g)->launches++;                                                         \
+  } while (0)
+
+inline unsigned grid_for(uint64_t n, int block = 256, int max_blocks = MAX_RESIDENT_BLOCKS) {
+  uint64_t b = (n + block - 1) / block;
+  if (b < 1) b = 1;
+  if (b > (uint64_t)max_blocks) b = max_blocks;
+  return (unsigned)b;
+}
+
+// allocate (stream-ordered) at least `bytes`, keeping the old block when large enough
+cudaError_t ensure(DevBuf &b, size_t bytes, cudaStream_t s);
+void release(DevBuf &b, cudaStream_t s);
+
+// exclusive scan: out[0..n) = prefix sums of in[0..n), out[n] = total.  in == out allowed.
+void scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s);
+void scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s);
+// stable LSD radix sort of (key, val) pairs on the given 8-bit digit shifts; returns
+// the index (0/1) of the buffer pair holding the result.
+int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1, uint64_t n,
+                     const int *shifts, int nshift, cudaStream_t s);
+// digit shifts covering the significant bits of keys with src, dst < V
+int key_shifts(uint32_t V, int *shifts);
+
+// thresholds (R4/R5) -- the library's own implementation (independent of oracle/)
+void level_bounds(uint32_t L, uint32_t h, uint32_t rho0, uint32_t rhoh, uint32_t tau0,
+                  uint32_t tauh, std::vector<uint64_t> &mn, std::vector<uint64_t> &mx);
+uint32_t leaf_rule(uint64_t cap0);
+inline uint32_t ilog2(uint64_t x) { uint32_t r = 0; while (x > 1) { x >>= 1; ++r; } return r; }
+
+gpma_status cuda_fail(gpma *g, cudaError_t e, const char *where);
+
+// update engine (update.cu)
+gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op,
+                         cudaStream_t s);
+gpma_status build_from_sorted(gpma *g, const uint64_t *sk, const uint32_t *sv, uint64_t m,
+                              cudaStream_t s);
+gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaStream_t s);
+gpma_status recompute_heads(gpma *g, cudaStream_t s);
+gpma_status count_slots(gpma *g, uint64_t *live_edges, uint64_t *tombs, cudaStream_t s);
+
+// analytics (analytics.cu)
+gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s);
+gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s);
+gpma_status pagerank_f64(gpma *g, double *x, int warm, double d, double tol, int max_iter, int *iters,
+                         cudaStream_t s);
+gpma_status pagerank_f32(gpma *g, float *x, int warm, float d, float tol, int max_iter, int *iters,
+                         cudaStream_t s);
+gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val, uint64_t cap_nnz,
+                       uint64_t *nnz_out, cudaStream_t s);
+
+}  // namespace gp
+
+#define GP_CHECK(g, call)                                   \
+  do {                                                      \
+    cudaError_t e_ = (call);                                \
+    if (e_ != cudaSuccess) return gp::cuda_fail((g), e_, #call); \
+  } while (0)

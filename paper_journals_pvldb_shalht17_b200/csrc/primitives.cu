@@ -1,0 +1,321 @@
+// primitives.cu -- scans, stable LSD radix sort, thresholds, memory helpers (sm_100a).
+//
+// Alg. 4 builds GPMA+ from standard GPU primitives (RunLengthEncoding,
+// ExclusiveScan; radix sort of the integer keys).  These are this
+// library's own implementations -- no CUB / Thrust.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+
+#include "gpma_internal.cuh"
+
+namespace gp {
+
+// ------------------------------------------------------------------ memory
+cudaError_t ensure(DevBuf &b, size_t bytes, cudaStream_t s) {
+  if (bytes == 0) bytes = 16;
+  if (b.bytes >= bytes) return cudaSuccess;
+  if (b.p) cudaFreeAsync(b.p, s);
+  b.p = nullptr;
+  b.bytes = 0;
+  size_t want = std::max(bytes, (size_t)(b.bytes * 3 / 2));
+  cudaError_t e = cudaMallocAsync(&b.p, want, s);
+  if (e != cudaSuccess) {
+    b.p = nullptr;
+    return e;
+  }
+  b.bytes = want;
+  return cudaSuccess;
+}
+
+void release(DevBuf &b, cudaStream_t s) {
+  if (b.p) cudaFreeAsync(b.p, s);
+  b.p = nullptr;
+  b.bytes = 0;
+}
+
+gpma_status cuda_fail(gpma *g, cudaError_t e, const char *where) {
+  if (e == cudaErrorMemoryAllocation) {
+    cudaGetLastError();
+    g->err = std::string("out of device memory in ") + where;
+    return GPMA_ERR_OOM;
+  }
+  g->poisoned = true;
+  g->err = std::string(cudaGetErrorString(e)) + " in " + where;
+  return GPMA_ERR_CUDA;
+}
+
+// ------------------------------------------------------------------ thresholds
+// R4: rho_i / tau_i linear in the level between the Fig. 3 leaf and root values
+// (P:417-422); R5: integer entry bounds capped at twice the child's bound.
+void level_bounds(uint32_t L, uint32_t h, uint32_t rho0, uint32_t rhoh, uint32_t tau0,
+                  uint32_t tauh, std::vector<uint64_t> &mn, std::vector<uint64_t> &mx) {
+  mn.assign(h + 1, 0);
+  mx.assign(h + 1, 0);
+  const uint64_t H = h ? h : 1;
+  for (uint32_t i = 0; i <= h; ++i) {
+    const uint64_t slots = (uint64_t)L << i;
+    const uint64_t wr = h ? (uint64_t)rho0 * (h - i) + (uint64_t)rhoh * i : rho0;
+    const uint64_t wt = h ? (uint64_t)tau0 * (h - i) + (uint64_t)tauh * i : tau0;
+    const uint64_t q = 10000ull * H;
+    uint64_t lo = (wr * slots) / q + ((wr * slots) % q != 0);  // ceil
+    uint64_t hi = (wt * slots) / q;                              // floor
+    if (i) {
+      lo = std::min(lo, 2 * mn[i - 1]);
+      hi = std::min(hi, 2 * mx[i - 1]);
+    }
+    mn[i] = lo;
+    mx[i] = hi;
+  }
+}
+
+// R3: leaf segment of O(log N) slots, a power of two: max(4, 2^floor(log2(log2 cap0))).
+uint32_t leaf_rule(uint64_t cap0) {
+  uint32_t lg = ilog2(cap0);
+  uint32_t L = 1u << ilog2(lg);
+  return L < 4 ? 4 : L;
+}
+
+int key_shifts(uint32_t V, int *shifts) {
+  uint32_t bits = V <= 1 ? 1 : ilog2((uint64_t)V - 1) + 1;
+  int n = 0;
+  for (uint32_t s = 0; s < bits; s += 8) shifts[n++] = (int)s;
+  for (uint32_t s = 0; s < bits; s += 8) shifts[n++] = (int)(32 + s);
+  return n;
+}
+
+// ------------------------------------------------------------------ scans
+constexpr int SC_THREADS = 256;
+constexpr int SC_ITEMS = 16;
+constexpr int SC_TILE = SC_THREADS * SC_ITEMS;   // 4096
+constexpr uint64_t SC_SINGLE_MAX = 1 << 16;
+
+template <typename T>
+__device__ __forceinline__ T warp_sum(T x) {
+#pragma unroll
+  for (int o = 16; o; o >>= 1) x += __shfl_xor_sync(0xffffffffu, x, o);
+  return x;
+}
+
+template <typename T>
+__device__ __forceinline__ T warp_incl_scan(T x, int lane) {
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    T y = __shfl_up_sync(0xffffffffu, x, o);
+    if (lane >= o) x += y;
+  }
+  return x;
+}
+
+template <typename T>
+__global__ void k_scan_single(const T *__restrict__ in, T *__restrict__ out, uint64_t n) {
+  __shared__ T wsum[32];
+  __shared__ T carry_s;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  if (threadIdx.x == 0) carry_s = 0;
+  __syncthreads();
+  for (uint64_t base = 0; base < n; base += blockDim.x) {
+    uint64_t i = base + threadIdx.x;
+    T x = i < n ? in[i] : T(0);
+    T inc = warp_incl_scan(x, lane);
+    if (lane == 31) wsum[w] = inc;
+    __syncthreads();
+    if (w == 0) {
+      T s = lane < (int)(blockDim.x >> 5) ? wsum[lane] : T(0);
+      T si = warp_incl_scan(s, lane);
+      wsum[lane] = si - s;
+    }
+    __syncthreads();
+    T c = carry_s;
+    if (i < n) out[i] = c + wsum[w] + inc - x;
+    __syncthreads();
+    if (threadIdx.x == blockDim.x - 1) carry_s = c + wsum[w] + inc;
+    __syncthreads();
+  }
+  if (threadIdx.x == 0) out[n] = carry_s;
+}
+
+template <typename T>
+__global__ void k_scan_reduce(const T *__restrict__ in, T *__restrict__ partial, uint64_t n) {
+  __shared__ T ws[SC_THREADS / 32];
+  const uint64_t base = (uint64_t)blockIdx.x * SC_TILE;
+  T s = 0;
+#pragma unroll
+  for (int j = 0; j < SC_ITEMS; ++j) {
+    uint64_t i = base + (uint64_t)j * SC_THREADS + threadIdx.x;
+    if (i < n) s += in[i];
+  }
+  s = warp_sum(s);
+  if ((threadIdx.x & 31) == 0) ws[threadIdx.x >> 5] = s;
+  __syncthreads();
+  if (threadIdx.x < 32) {
+    T t = threadIdx.x < SC_THREADS / 32 ? ws[threadIdx.x] : T(0);
+    t = warp_sum(t);
+    if (threadIdx.x == 0) partial[blockIdx.x] = t;
+  }
+}
+
+template <typename T>
+__global__ void k_scan_down(const T *in, T *out, const T *__restrict__ partial, uint64_t n,
+                            uint64_t nb) {
+  __shared__ T ws[SC_THREADS / 32];
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  const uint64_t base = (uint64_t)blockIdx.x * SC_TILE + (uint64_t)w * (32 * SC_ITEMS);
+  T s = 0;
+#pragma unroll
+  for (int j = 0; j < SC_ITEMS; ++j) {
+    uint64_t i = base + j * 32 + lane;
+    if (i < n) s += in[i];
+  }
+  s = warp_sum(s);
+  if (lane == 0) ws[w] = s;
+  __syncthreads();
+  T carry = partial[blockIdx.x];
+  for (int k = 0; k < w; ++k) carry += ws[k];
+#pragma unroll
+  for (int j = 0; j < SC_ITEMS; ++j) {
+    uint64_t i = base + j * 32 + lane;
+    T x = i < n ? in[i] : T(0);
+    T inc = warp_incl_scan(x, lane);
+    if (i < n) out[i] = carry + inc - x;
+    carry += __shfl_sync(0xffffffffu, inc, 31);
+  }
+  if (blockIdx.x == 0 && threadIdx.x == 0) out[n] = partial[nb];
+}
+
+template <typename T>
+static void scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s, T *tmp) {
+  if (n <= SC_SINGLE_MAX) {
+    GP_LAUNCH(g, k_scan_single<T>, 1, 1024, 0, s, in, out, n);
+    return;
+  }
+  uint64_t nb = (n + SC_TILE - 1) / SC_TILE;
+  T *partial = tmp;
+  GP_LAUNCH(g, k_scan_reduce<T>, (unsigned)nb, SC_THREADS, 0, s, in, partial, n);
+  scan_impl<T>(g, partial, partial, nb, s, tmp + nb + 1);
+  GP_LAUNCH(g, k_scan_down<T>, (unsigned)nb, SC_THREADS, 0, s, in, out, partial, n, nb);
+}
+
+static size_t scan_tmp_elems(uint64_t n) {
+  size_t t = 0;
+  while (n > SC_SINGLE_MAX) {
+    n = (n + SC_TILE - 1) / SC_TILE;
+    t += n + 1;
+  }
+  return t + 1;
+}
+
+void scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s) {
+  ensure(g->b_scan, scan_tmp_elems(n) * sizeof(uint64_t), s);
+  scan_impl<uint32_t>(g, in, out, n, s, (uint32_t *)g->b_scan.p);
+}
+
+void scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s) {
+  ensure(g->b_scan, scan_tmp_elems(n) * sizeof(uint64_t), s);
+  scan_impl<uint64_t>(g, in, out, n, s, (uint64_t *)g->b_scan.p);
+}
+
+// ------------------------------------------------------------------ radix sort
+// Stable LSD radix sort, 8-bit digits, only over the significant key bits (the
+// u64 key is src<<32|dst with src,dst < V).  Per pass: tile histograms -> one
+// exclusive scan over the digit-major (digit, tile) table -> stable scatter, where
+// the rank inside a tile comes from __match_any_sync peer groups per warp round.
+constexpr int RS_THREADS = 256;
+constexpr int RS_ITEMS = 16;
+constexpr int RS_WARPS = RS_THREADS / 32;
+constexpr int RS_TILE = RS_THREADS * RS_ITEMS;
+
+__global__ void __launch_bounds__(RS_THREADS) k_radix_hist(const uint64_t *__restrict__ keys,
+                                                           uint64_t n, int shift,
+                                                           uint32_t *__restrict__ hist,
+                                                           uint32_t ntiles) {
+  __shared__ uint32_t h[256];
+  h[threadIdx.x] = 0;
+  __syncthreads();
+  const uint64_t base = (uint64_t)blockIdx.x * RS_TILE;
+#pragma unroll 4
+  for (int j = 0; j < RS_ITEMS; ++j) {
+    uint64_t i = base + (uint64_t)j * RS_THREADS + threadIdx.x;
+    if (i < n) atomicAdd(&h[(keys[i] >> shift) & 255u], 1u);
+  }
+  __syncthreads();
+  hist[(uint64_t)threadIdx.x * ntiles + blockIdx.x] = h[threadIdx.x];
+}
+
+__global__ void __launch_bounds__(RS_THREADS) k_radix_scatter(
+    const uint64_t *__restrict__ kin, const uint32_t *__restrict__ vin, uint64_t *__restrict__ kout,
+    uint32_t *__restrict__ vout, uint64_t n, int shift, const uint32_t *__restrict__ hscan,
+    uint32_t ntiles) {
+  __shared__ uint32_t wc[RS_WARPS][256];
+  for (int d = threadIdx.x; d < RS_WARPS * 256; d += RS_THREADS) (&wc[0][0])[d] = 0;
+  __syncthreads();
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint64_t base = (uint64_t)blockIdx.x * RS_TILE + (uint64_t)w * (32 * RS_ITEMS);
+  uint64_t k[RS_ITEMS];
+  uint32_t v[RS_ITEMS], r[RS_ITEMS];
+#pragma unroll
+  for (int j = 0; j < RS_ITEMS; ++j) {
+    uint64_t i = base + j * 32 + lane;
+    bool ok = i < n;
+    k[j] = ok ? kin[i] : 0;
+    v[j] = ok ? vin[i] : 0;
+  }
+#pragma unroll
+  for (int j = 0; j < RS_ITEMS; ++j) {
+    uint64_t i = base + j * 32 + lane;
+    bool ok = i < n;
+    uint32_t d = ok ? (uint32_t)(k[j] >> shift) & 255u : 256u + lane;
+    uint32_t peers = __match_any_sync(0xffffffffu, d);
+    uint32_t cur = ok ? wc[w][d] : 0u;
+    __syncwarp();
+    uint32_t rank = __popc(peers & lt);
+    if (ok && rank == 0) wc[w][d] = cur + __popc(peers);
+    __syncwarp();
+    r[j] = cur + rank;
+  }
+  __syncthreads();
+  {
+    int d = threadIdx.x;  // 256 threads == 256 digits
+    uint32_t run = 0;
+#pragma unroll
+    for (int ww = 0; ww < RS_WARPS; ++ww) {
+      uint32_t t = wc[ww][d];
+      wc[ww][d] = run;
+      run += t;
+    }
+  }
+  __syncthreads();
+#pragma unroll
+  for (int j = 0; j < RS_ITEMS; ++j) {
+    uint64_t i = base + j * 32 + lane;
+    if (i < n) {
+      uint32_t d = (uint32_t)(k[j] >> shift) & 255u;
+      uint64_t pos = (uint64_t)hscan[(uint64_t)d * ntiles + blockIdx.x] + wc[w][d] + r[j];
+      kout[pos] = k[j];
+      vout[pos] = v[j];
+    }
+  }
+}
+
+int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1, uint64_t n,
+                     const int *shifts, int nshift, cudaStream_t s) {
+  if (n <= 1) return 0;
+  const uint32_t ntiles = (uint32_t)((n + RS_TILE - 1) / RS_TILE);
+  const uint64_t hn = (uint64_t)ntiles * 256;
+  ensure(g->b_hist, (hn + 1) * sizeof(uint32_t), s);
+  uint32_t *hist = (uint32_t *)g->b_hist.p;
+  uint64_t *ks[2] = {k0, k1};
+  uint32_t *vs[2] = {v0, v1};
+  int cur = 0;
+  for (int p = 0; p < nshift; ++p) {
+    GP_LAUNCH(g, k_radix_hist, ntiles, RS_THREADS, 0, s, ks[cur], n, shifts[p], hist, ntiles);
+    scan_u32(g, hist, hist, hn, s);
+    GP_LAUNCH(g, k_radix_scatter, ntiles, RS_THREADS, 0, s, ks[cur], vs[cur], ks[cur ^ 1],
+              vs[cur ^ 1], n, shifts[p], hist, ntiles);
+    cur ^= 1;
+  }
+  return cur;
+}
+
+}  // namespace gp

@@ -1,0 +1,952 @@
+// update.cu -- GPMA+ batch update on sm_100a (Alg. 4).
+//
+// Per batch:  validate -> Sort(U) (l.2, radix sort of the integer keys)
+//   -> unique (last occurrence wins, R10) -> BinarySearchLeafSegments (l.3, R9)
+//   -> pre-pass: overwrite / revive / lazy-delete in place
+//   -> level loop i = 0..h (l.4-15): UniqueSegments = RLE + ExclusiveScan (l.18-21),
+//      CountSegment + CountUpdatesInSegment + density test (l.23-25, R5 integer
+//      bounds), Merge + re-dispatch evenly (l.26-27, R7 proportional split), promote
+//      the rest to the parent segment (l.12-15)
+//   -> root resize (l.16-17, R14) -> locate-index (head) fix-up.
+//
+// Data layout in HBM: key u64[cap] and val u32[cap] as two
+// SoA arrays (16-B vector moves on both), live count u32 per leaf, head u64 per leaf,
+// row_offset u64[V+1].  Every window is rewritten out of place through a dense scratch
+// list (gather -> scatter), so no kernel ever reads a slot another CTA writes.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+
+#include "gpma_internal.cuh"
+
+namespace gp {
+
+constexpr int TB = 256;
+
+__device__ __forceinline__ uint32_t locate_leaf(const uint64_t *__restrict__ head, uint32_t nleaves,
+                                                uint64_t k) {
+  // R9: upper_bound over the monotone head array, minus one, clamped at leaf 0.
+  uint32_t lo = 0, hi = nleaves;
+  while (lo < hi) {
+    uint32_t mid = (lo + hi) >> 1;
+    if (__ldg(head + mid) <= k) lo = mid + 1;
+    else hi = mid;
+  }
+  return lo ? lo - 1 : 0;
+}
+
+// ------------------------------------------------------------------ validate
+__global__ void k_validate(const uint64_t *__restrict__ keys, const uint32_t *__restrict__ vals,
+                           uint64_t n, uint32_t V, int check_vals, Ctrl *c) {
+  uint32_t e = 0;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t k = keys[i];
+    uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
+    if (dst == COL_GUARD) e |= 2u;
+    if (check_vals && vals[i] == VAL_TOMB) e |= 2u;
+    if (src >= V || dst >= V) e |= 1u;
+  }
+  e = __reduce_or_sync(0xffffffffu, e);
+  if (e && (threadIdx.x & 31) == 0) atomicOr(&c->err, e);
+}
+
+// ------------------------------------------------------------------ pre-pass
+// One thread per sorted update; only the last copy of a key acts (R10).
+__global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__restrict__ sv,
+                          uint64_t n, const uint64_t *__restrict__ key, uint32_t *__restrict__ val,
+                          uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
+                          uint32_t nleaves, uint32_t L, int op, int mode,
+                          uint32_t *__restrict__ keep, uint32_t *__restrict__ tgt, Ctrl *c) {
+  uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
+  uint32_t uniq = 0;
+  if (i < n) {
+    uint64_t k = sk[i];
+    uint32_t kp = 0, t = 0;
+    if (i + 1 == n || sk[i + 1] != k) {
+      uniq = 1;
+      t = locate_leaf(head, nleaves, k);
+      uint64_t base = (uint64_t)t * L, hit = KEY_NONE;
+      for (uint32_t p = 0; p < L; ++p) {
+        uint64_t x = key[base + p];
+        if (x == k) { hit = base + p; break; }
+        if (x == KEY_NONE || x > k) break;
+      }
+      if (op == GPMA_INSERT) {
+        if (hit != KEY_NONE) {                      // overwrite (R11) or revive (R12)
+          uint32_t old = val[hit];
+          val[hit] = sv[i];
+          if (old == VAL_TOMB) atomicAdd(&cnt[t], 1u);
+        } else {
+          kp = 1;
+        }
+      } else if (mode == GPMA_DELETE_LAZY) {        // mark, no maintenance
+        if (hit != KEY_NONE && val[hit] != VAL_TOMB) {
+          val[hit] = VAL_TOMB;
+          atomicSub(&cnt[t], 1u);
+        }
+      } else {                                      // strict delete: live keys only
+        if (hit != KEY_NONE && val[hit] != VAL_TOMB) kp = 1;
+      }
+    }
+    keep[i] = kp;
+    tgt[i] = t;
+  }
+  uint32_t u = __reduce_add_sync(0xffffffffu, uniq);
+  if ((threadIdx.x & 31) == 0 && u) atomicAdd((unsigned long long *)&c->nunique, (unsigned long long)u);
+}
+
+__global__ void k_compact_pending(const uint32_t *__restrict__ keep, const uint32_t *__restrict__ pos,
+                                  uint64_t n, const uint64_t *__restrict__ ik,
+                                  const uint32_t *__restrict__ iv, const uint32_t *__restrict__ it,
+                                  uint64_t *__restrict__ ok, uint32_t *__restrict__ ov,
+                                  uint32_t *__restrict__ ot) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    if (keep[i]) {
+      uint32_t d = pos[i];
+      ok[d] = ik[i];
+      ov[d] = iv[i];
+      ot[d] = it[i];
+    }
+  }
+}
+
+// ------------------------------------------------------------------ level step
+struct Lvl {
+  const uint64_t *pk;
+  const uint32_t *pv;
+  const uint32_t *pt;
+  uint64_t p;          // pending entering this level (host-known)
+  uint32_t lvl;        // tree level i
+  uint32_t L;
+  uint32_t *hf, *widx, *wfirst, *acc, *aidx, *alist, *keep, *kpos;
+  uint64_t *nw, *woff, *lpre;
+  uint64_t *wk;        // scratch: merged windows, dense
+  uint32_t *wv;
+  uint64_t tmin, tmax;
+  int op;
+  int force;           // resize: accept the single root window unconditionally
+};
+
+__global__ void k_lvl_flags(Lvl a) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < a.p;
+       j += (uint64_t)gridDim.x * blockDim.x)
+    a.hf[j] = (j == 0 || (a.pt[j] >> a.lvl) != (a.pt[j - 1] >> a.lvl)) ? 1u : 0u;
+}
+
+__global__ void k_lvl_first(Lvl a) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < a.p;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    if (a.hf[j]) a.wfirst[a.widx[j]] = (uint32_t)j;
+    if (j == 0) a.wfirst[a.widx[a.p]] = (uint32_t)a.p;
+  }
+}
+
+// CountSegment + CountUpdatesInSegment + density test (Alg. 4 l.23-25).
+// TPW threads per window sum the per-leaf live counts of the window.
+template <int TPW>
+__global__ void k_lvl_count(Lvl a, const uint32_t *__restrict__ cnt) {
+  __shared__ uint64_t red[TB / 32];
+  const uint32_t q = a.widx[a.p];
+  const uint64_t groups_per_grid = (uint64_t)gridDim.x * (blockDim.x / TPW);
+  const uint64_t g0 = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / TPW;
+  const int r = threadIdx.x % TPW;
+  const uint64_t nleaf_w = 1ull << a.lvl;
+  // the loop trip count must be uniform inside a group
+  for (uint64_t w = g0; w < a.p; w += groups_per_grid) {
+    uint64_t n = 0;
+    bool real = w < q;
+    uint64_t leaf0 = 0;
+    if (real) {
+      leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+      for (uint64_t l = r; l < nleaf_w; l += TPW) n += cnt[leaf0 + l];
+    }
+    if (TPW >= 32) {
+      for (int o = 16; o; o >>= 1) n += __shfl_xor_sync(0xffffffffu, n, o);
+      if (TPW > 32) {
+        if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = n;
+        __syncthreads();
+        if (threadIdx.x == 0) {
+          uint64_t s = 0;
+          for (int k = 0; k < TPW / 32; ++k) s += red[k];
+          red[0] = s;
+        }
+        __syncthreads();
+        n = red[0];
+        __syncthreads();
+      }
+    }
+    if (r == 0) {
+      if (!real) {
+        a.acc[w] = 0;
+        a.nw[w] = 0;
+      } else {
+        uint64_t u = a.wfirst[w + 1] - a.wfirst[w];
+        bool ok;
+        if (a.force) ok = true;
+        else if (a.op == GPMA_INSERT) ok = n + u <= a.tmax;
+        else ok = n >= u && n - u >= a.tmin;
+        a.acc[w] = ok ? 1u : 0u;
+        a.nw[w] = ok ? (a.op == GPMA_INSERT ? n + u : n - u) : 0;
+      }
+    }
+  }
+}
+
+__global__ void k_lvl_alist(Lvl a) {
+  for (uint64_t w = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; w < a.p;
+       w += (uint64_t)gridDim.x * blockDim.x)
+    if (a.acc[w]) a.alist[a.aidx[w]] = (uint32_t)w;
+}
+
+// live counts of the leaves of the accepted windows, flattened (then scanned)
+__global__ void k_lvl_leafcnt(Lvl a, const uint32_t *__restrict__ cnt, uint64_t bound) {
+  const uint32_t nacc = a.aidx[a.p];
+  const uint64_t mask = (1ull << a.lvl) - 1;
+  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < bound;
+       g += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t ai = g >> a.lvl;
+    uint64_t v = 0;
+    if (ai < nacc) {
+      uint32_t w = a.alist[ai];
+      uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+      v = cnt[leaf0 + (g & mask)];
+    }
+    a.lpre[g] = v;
+  }
+}
+
+__device__ __forceinline__ uint64_t lower_bound_u64(const uint64_t *__restrict__ x, uint64_t lo,
+                                                    uint64_t hi, uint64_t k) {
+  while (lo < hi) {
+    uint64_t mid = (lo + hi) >> 1;
+    if (x[mid] < k) lo = mid + 1;
+    else hi = mid;
+  }
+  return lo;
+}
+
+// Gather the live entries of every accepted window into the dense scratch list at
+// their merged rank (Merge, Alg. 4 l.26).  Tombstones are dropped (R12).  Threads
+// map to slots; a leaf never straddles a warp (L | 32), so ballots rank inside it.
+__global__ void k_lvl_gather(Lvl a, const uint64_t *__restrict__ key, const uint32_t *__restrict__ val,
+                             uint64_t bound_r) {
+  const uint32_t nacc = a.aidx[a.p];
+  const uint64_t wslots = (uint64_t)a.L << a.lvl;
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint32_t leafmask = (a.L == 32 ? 0xffffffffu : ((1u << a.L) - 1u) << (lane & ~(a.L - 1)));
+  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < bound_r;
+       g += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t ai = g / wslots;
+    bool valid = ai < nacc;
+    uint64_t k = KEY_NONE, s = 0;
+    uint32_t v = 0, w = 0;
+    if (valid) {
+      w = a.alist[ai];
+      uint64_t seg = a.pt[a.wfirst[w]] >> a.lvl;
+      s = seg * wslots + (g % wslots);
+      k = key[s];
+      v = val[s];
+    }
+    bool live = valid && k != KEY_NONE && v != VAL_TOMB;
+    uint32_t bal = __ballot_sync(0xffffffffu, live);
+    if (live) {
+      uint64_t off = g % wslots;
+      uint64_t lidx = off / a.L;
+      uint64_t rl = __popc(bal & leafmask & lt);
+      if (a.lvl) rl += a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl];
+      uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
+      uint64_t c = lower_bound_u64(a.pk, ub, ue, k) - ub;
+      uint64_t r;
+      bool drop = false;
+      if (a.op == GPMA_INSERT) {
+        r = rl + c;
+      } else {
+        drop = (ub + c < ue) && a.pk[ub + c] == k;
+        r = rl - c;
+      }
+      if (!drop) {
+        uint64_t d = a.woff[w] + r;
+        a.wk[d] = k;
+        a.wv[d] = v;
+      }
+    }
+  }
+}
+
+// Place the pending insertions of accepted windows at their merged rank.
+__global__ void k_lvl_place(Lvl a, const uint64_t *__restrict__ key, const uint32_t *__restrict__ val) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < a.p;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t w = a.widx[j] + a.hf[j] - 1;
+    if (!a.acc[w]) continue;
+    uint64_t ai = a.aidx[w];
+    uint32_t t = a.pt[j];
+    uint64_t k = a.pk[j];
+    uint64_t seg = t >> a.lvl;
+    uint64_t lidx = t - (seg << a.lvl);
+    uint64_t rl = a.lvl ? a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl] : 0;
+    uint64_t base = (uint64_t)t * a.L;
+    for (uint32_t p = 0; p < a.L; ++p) {
+      uint64_t x = key[base + p];
+      if (x == KEY_NONE || x > k) break;
+      if (val[base + p] != VAL_TOMB) ++rl;
+    }
+    uint64_t d = a.woff[w] + (j - a.wfirst[w]) + rl;
+    a.wk[d] = k;
+    a.wv[d] = a.pv[j];
+  }
+}
+
+// Re-dispatch evenly (Alg. 4 l.27, R7): leaf l of a window with Lc leaves and N
+// entries receives entries [floor(l N / Lc), floor((l+1) N / Lc)), left-packed.
+// Guards moved here update the row offsets (R8).
+__global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
+                                   uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset,
+                                   uint64_t bound, uint2 *__restrict__ dirty, uint64_t dirty_base) {
+  const uint32_t nacc = a.aidx[a.p];
+  const uint64_t Lc = 1ull << a.lvl;
+  const uint64_t wslots = (uint64_t)a.L << a.lvl;
+  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < bound;
+       g += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t ai = g / wslots;
+    if (ai >= nacc) continue;
+    uint32_t w = a.alist[ai];
+    uint64_t N = a.nw[w];
+    uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+    uint64_t off = g % wslots;
+    uint64_t l = off / a.L, p = off % a.L;
+    uint64_t lo = l * N / Lc, hi = (l + 1) * N / Lc;
+    uint64_t s = leaf0 * a.L + off;
+    if (p < hi - lo) {
+      uint64_t e = a.woff[w] + lo + p;
+      uint64_t k = a.wk[e];
+      key[s] = k;
+      val[s] = a.wv[e];
+      if (is_guard_key(k)) row_offset[(k >> 32) + 1] = s;
+    } else {
+      key[s] = KEY_NONE;
+      val[s] = 0;
+    }
+    if (p == 0) cnt[leaf0 + l] = (uint32_t)(hi - lo);
+    if (off == 0) dirty[dirty_base + ai] = make_uint2((uint32_t)leaf0, (uint32_t)Lc);
+  }
+}
+
+__global__ void k_lvl_keep(Lvl a) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < a.p;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t w = a.widx[j] + a.hf[j] - 1;
+    a.keep[j] = a.acc[w] ? 0u : 1u;
+  }
+}
+
+__global__ void k_lvl_summary(Lvl a, Ctrl *c) {
+  // sum  = unique windows | accepted windows << 32 ; sum2 = pending after this level
+  c->sum = (uint64_t)a.widx[a.p] | ((uint64_t)a.aidx[a.p] << 32);
+  c->sum2 = a.kpos[a.p];
+}
+
+// Whole-array even layout of a dense sorted list (create, resize; R7 over all leaves).
+__global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *__restrict__ wv,
+                              uint64_t N, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
+                              uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset,
+                              uint32_t L, uint64_t nleaves) {
+  const uint64_t cap = nleaves * L;
+  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
+       s += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t l = s / L, p = s % L;
+    uint64_t lo = l * N / nleaves, hi = (l + 1) * N / nleaves;
+    if (p < hi - lo) {
+      uint64_t k = wk[lo + p];
+      key[s] = k;
+      val[s] = wv[lo + p];
+      if (is_guard_key(k)) row_offset[(k >> 32) + 1] = s;
+    } else {
+      key[s] = KEY_NONE;
+      val[s] = 0;
+    }
+    if (p == 0) cnt[l] = (uint32_t)(hi - lo);
+  }
+}
+
+// ------------------------------------------------------------------ locate index
+__device__ __forceinline__ uint64_t next_head(const uint64_t *__restrict__ key, uint32_t L,
+                                              uint64_t nleaves, uint64_t l) {
+  for (; l < nleaves; ++l) {
+    uint64_t k = key[l * L];
+    if (k != KEY_NONE) return k;
+  }
+  return KEY_NONE;
+}
+
+// head[l] = first key of the first non-empty leaf >= l (KEY_NONE if none): a pure
+// function of the layout, so concurrent writers agree.
+__global__ void k_heads_all(const uint64_t *__restrict__ key, uint64_t *__restrict__ head, uint32_t L,
+                            uint64_t nleaves) {
+  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
+       l += (uint64_t)gridDim.x * blockDim.x)
+    head[l] = next_head(key, L, nleaves, l);
+}
+
+// Fix the heads of rewritten windows and of the run of empty leaves left of them.
+__global__ void k_heads_dirty(const uint64_t *__restrict__ key, uint64_t *__restrict__ head,
+                              uint32_t L, uint64_t nleaves, const uint2 *__restrict__ dirty,
+                              uint64_t ndirty) {
+  const int lane = threadIdx.x & 31;
+  const uint64_t warps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  for (uint64_t d = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32; d < ndirty; d += warps) {
+    uint2 wd = dirty[d];
+    for (uint64_t l = wd.x + lane; l < (uint64_t)wd.x + wd.y; l += 32)
+      head[l] = next_head(key, L, nleaves, l);
+    if (lane == 0) {
+      uint64_t hv = next_head(key, L, nleaves, wd.x);
+      for (int64_t m = (int64_t)wd.x - 1; m >= 0 && key[(uint64_t)m * L] == KEY_NONE; --m) head[m] = hv;
+    }
+  }
+}
+
+__global__ void k_sum_cnt(const uint32_t *__restrict__ cnt, uint64_t nleaves, Ctrl *c) {
+  uint64_t s = 0;
+  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
+       l += (uint64_t)gridDim.x * blockDim.x)
+    s += cnt[l];
+  for (int o = 16; o; o >>= 1) s += __shfl_xor_sync(0xffffffffu, s, o);
+  if ((threadIdx.x & 31) == 0 && s) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)s);
+}
+
+__global__ void k_count_slots(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val,
+                              uint64_t cap, Ctrl *c) {
+  uint64_t e = 0, t = 0;
+  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
+       s += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t k = key[s];
+    if (k == KEY_NONE || is_guard_key(k)) continue;
+    if (val[s] == VAL_TOMB) ++t;
+    else ++e;
+  }
+  for (int o = 16; o; o >>= 1) {
+    e += __shfl_xor_sync(0xffffffffu, e, o);
+    t += __shfl_xor_sync(0xffffffffu, t, o);
+  }
+  if ((threadIdx.x & 31) == 0) {
+    if (e) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)e);
+    if (t) atomicAdd((unsigned long long *)&c->sum2, (unsigned long long)t);
+  }
+}
+
+// create: merge sorted unique edges with the V guards into a dense list (R1).
+// Edge j with source u lands at j + u; guard u at (#edges with src <= u) + u.
+__global__ void k_place_edges(const uint64_t *__restrict__ sk, const uint32_t *__restrict__ sv,
+                              const uint32_t *__restrict__ pos, const uint32_t *__restrict__ keep,
+                              uint64_t n, uint64_t *__restrict__ wk, uint32_t *__restrict__ wv) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    if (!keep[i]) continue;
+    uint64_t k = sk[i];
+    uint64_t d = (uint64_t)pos[i] + (k >> 32);
+    wk[d] = k;
+    wv[d] = sv[i];
+  }
+}
+
+__global__ void k_place_guards(const uint64_t *__restrict__ wk_edges_sorted_unused, uint32_t V,
+                               const uint64_t *__restrict__ ek, uint64_t m, uint64_t *__restrict__ wk,
+                               uint32_t *__restrict__ wv) {
+  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < V;
+       u += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t gk = (u << 32) | COL_GUARD;
+    // number of edges with key < guard key, searched in the dense edge list ek[0..m)
+    uint64_t lo = 0, hi = m;
+    while (lo < hi) {
+      uint64_t mid = (lo + hi) >> 1;
+      if (ek[mid] < gk) lo = mid + 1;
+      else hi = mid;
+    }
+    wk[lo + u] = gk;
+    wv[lo + u] = 0;
+  }
+}
+
+__global__ void k_unique_last(const uint64_t *__restrict__ sk, uint64_t n, uint32_t *__restrict__ keep) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x)
+    keep[i] = (i + 1 == n || sk[i + 1] != sk[i]) ? 1u : 0u;
+}
+
+__global__ void k_compact_kv(const uint32_t *__restrict__ keep, const uint32_t *__restrict__ pos,
+                             uint64_t n, const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
+                             uint64_t *__restrict__ ok, uint32_t *__restrict__ ov) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x)
+    if (keep[i]) {
+      ok[pos[i]] = ik[i];
+      ov[pos[i]] = iv[i];
+    }
+}
+
+__global__ void k_raw_counts(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val,
+                             uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset, uint32_t L,
+                             uint64_t nleaves, uint32_t V) {
+  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
+       l += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t c = 0;
+    for (uint32_t p = 0; p < L; ++p) {
+      uint64_t s = l * L + p;
+      uint64_t k = key[s];
+      if (k == KEY_NONE) continue;
+      if (val[s] != VAL_TOMB) ++c;
+      if (is_guard_key(k) && (k >> 32) < V) row_offset[(k >> 32) + 1] = s;
+    }
+    cnt[l] = c;
+  }
+}
+
+// ------------------------------------------------------------------ host driver
+static gpma_status read_ctrl(gpma *g, cudaStream_t s) {
+  GP_CHECK(g, cudaMemcpyAsync(g->ctrl_h, g->ctrl_d, sizeof(Ctrl), cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  return GPMA_OK;
+}
+
+static gpma_status zero_ctrl(gpma *g, cudaStream_t s) {
+  GP_CHECK(g, cudaMemsetAsync(g->ctrl_d, 0, sizeof(Ctrl), s));
+  return GPMA_OK;
+}
+
+gpma_status recompute_heads(gpma *g, cudaStream_t s) {
+  uint64_t nl = g->cap / g->L;
+  GP_LAUNCH(g, k_heads_all, grid_for(nl), TB, 0, s, g->key, g->head, g->L, nl);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+gpma_status count_slots(gpma *g, uint64_t *live_edges, uint64_t *tombs, cudaStream_t s) {
+  gpma_status st = zero_ctrl(g, s);
+  if (st) return st;
+  GP_LAUNCH(g, k_count_slots, grid_for(g->cap), TB, 0, s, g->key, g->val, g->cap, g->ctrl_d);
+  if ((st = read_ctrl(g, s))) return st;
+  *live_edges = g->ctrl_h->sum;
+  *tombs = g->ctrl_h->sum2;
+  return GPMA_OK;
+}
+
+static void set_geometry(gpma *g, uint64_t cap) {
+  g->cap = cap;
+  g->h = ilog2(cap / g->L);
+  level_bounds(g->L, g->h, g->rho0, g->rhoh, g->tau0, g->tauh, g->tmin, g->tmax);
+}
+
+static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v, uint32_t **c,
+                               uint64_t **hd, cudaStream_t s) {
+  uint64_t nl = cap / g->L;
+  *k = nullptr; *v = nullptr; *c = nullptr; *hd = nullptr;
+  cudaError_t e1 = cudaMallocAsync((void **)k, cap * 8, s);
+  cudaError_t e2 = cudaMallocAsync((void **)v, cap * 4, s);
+  cudaError_t e3 = cudaMallocAsync((void **)c, nl * 4, s);
+  cudaError_t e4 = cudaMallocAsync((void **)hd, nl * 8, s);
+  if (e1 || e2 || e3 || e4) {
+    cudaGetLastError();
+    if (*k) cudaFreeAsync(*k, s);
+    if (*v) cudaFreeAsync(*v, s);
+    if (*c) cudaFreeAsync(*c, s);
+    if (*hd) cudaFreeAsync(*hd, s);
+    g->err = "out of device memory allocating the store";
+    return GPMA_ERR_OOM;
+  }
+  return GPMA_OK;
+}
+
+// dense sorted list (wk, wv)[0..N) -> whole array of `cap` slots
+gpma_status build_from_sorted(gpma *g, const uint64_t *wk, const uint32_t *wv, uint64_t N,
+                              cudaStream_t s) {
+  uint64_t nl = g->cap / g->L;
+  GP_LAUNCH(g, k_layout_even, grid_for(g->cap), TB, 0, s, wk, wv, N, g->key, g->val, g->cnt,
+            g->row_offset, g->L, nl);
+  GP_CHECK(g, cudaGetLastError());
+  return recompute_heads(g, s);
+}
+
+gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaStream_t s) {
+  GP_CHECK(g, cudaMemcpyAsync(g->key, keys, g->cap * 8, cudaMemcpyDefault, s));
+  GP_CHECK(g, cudaMemcpyAsync(g->val, vals, g->cap * 4, cudaMemcpyDefault, s));
+  uint64_t nl = g->cap / g->L;
+  GP_LAUNCH(g, k_raw_counts, grid_for(nl), TB, 0, s, g->key, g->val, g->cnt, g->row_offset, g->L, nl,
+            g->V);
+  GP_CHECK(g, cudaGetLastError());
+  return recompute_heads(g, s);
+}
+
+// Sort a device batch (keys, vals) of n pairs and drop all but the last copy of each
+// key; returns the number of unique keys in *m, result in b_sk[0]/b_sv[0].
+static gpma_status sort_unique(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
+                               uint64_t *m, bool need_unique_compact, int *which, cudaStream_t s) {
+  GP_CHECK(g, ensure(g->b_sk[0], n * 8, s));
+  GP_CHECK(g, ensure(g->b_sk[1], n * 8, s));
+  GP_CHECK(g, ensure(g->b_sv[0], n * 4, s));
+  GP_CHECK(g, ensure(g->b_sv[1], n * 4, s));
+  uint64_t *k0 = (uint64_t *)g->b_sk[0].p, *k1 = (uint64_t *)g->b_sk[1].p;
+  uint32_t *v0 = (uint32_t *)g->b_sv[0].p, *v1 = (uint32_t *)g->b_sv[1].p;
+  GP_CHECK(g, cudaMemcpyAsync(k0, keys, n * 8, cudaMemcpyDefault, s));
+  if (vals) GP_CHECK(g, cudaMemcpyAsync(v0, vals, n * 4, cudaMemcpyDefault, s));
+  else GP_CHECK(g, cudaMemsetAsync(v0, 0, n * 4, s));
+  int sh[8];
+  int ns = key_shifts(g->V, sh);
+  *which = radix_sort_pairs(g, k0, v0, k1, v1, n, sh, ns, s);
+  (void)need_unique_compact;
+  *m = n;
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+static gpma_status validate(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
+                            bool check_vals, cudaStream_t s) {
+  gpma_status st = zero_ctrl(g, s);
+  if (st) return st;
+  GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, keys, vals, n, g->V, check_vals ? 1 : 0, g->ctrl_d);
+  if ((st = read_ctrl(g, s))) return st;
+  if (g->ctrl_h->err & 2u) return GPMA_ERR_RESERVED;
+  if (g->ctrl_h->err & 1u) return GPMA_ERR_RANGE;
+  return GPMA_OK;
+}
+
+gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
+                              uint64_t cap_override, uint32_t leaf_override, cudaStream_t s) {
+  gpma_status st;
+  uint64_t m = 0;
+  const uint64_t *ek = nullptr;
+  const uint32_t *ev = nullptr;
+  if (n) {
+    // stage + validate on device
+    GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
+    GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
+    GP_CHECK(g, cudaMemcpyAsync(g->b_stage[0].p, keys, n * 8, cudaMemcpyDefault, s));
+    GP_CHECK(g, cudaMemcpyAsync(g->b_stage[1].p, vals, n * 4, cudaMemcpyDefault, s));
+    if ((st = validate(g, (uint64_t *)g->b_stage[0].p, (uint32_t *)g->b_stage[1].p, n, true, s)))
+      return st;
+    int which;
+    uint64_t mm;
+    if ((st = sort_unique(g, (uint64_t *)g->b_stage[0].p, (uint32_t *)g->b_stage[1].p, n, &mm, true,
+                          &which, s)))
+      return st;
+    uint64_t *sk = (uint64_t *)g->b_sk[which].p;
+    uint32_t *sv = (uint32_t *)g->b_sv[which].p;
+    GP_CHECK(g, ensure(g->b_keep, (n + 1) * 4, s));
+    GP_CHECK(g, ensure(g->b_pos, (n + 1) * 4, s));
+    uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p;
+    GP_LAUNCH(g, k_unique_last, grid_for(n), TB, 0, s, sk, n, keep);
+    scan_u32(g, keep, pos, n, s);
+    uint32_t mh = 0;
+    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, pos + n, 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaStreamSynchronize(s));
+    mh = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
+    m = mh;
+    // dense unique edges into the other buffer
+    uint64_t *uk = (uint64_t *)g->b_sk[which ^ 1].p;
+    uint32_t *uv = (uint32_t *)g->b_sv[which ^ 1].p;
+    GP_LAUNCH(g, k_compact_kv, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, uk, uv);
+    ek = uk;
+    ev = uv;
+  }
+  const uint64_t E = m + g->V;
+  uint64_t cap;
+  if (cap_override) {
+    cap = cap_override;
+    g->L = leaf_override ? leaf_override : leaf_rule(cap);
+  } else {
+    cap = 8;
+    while (E > cap * g->init_bp / 10000) cap *= 2;
+    g->L = leaf_override ? leaf_override : leaf_rule(cap);
+    if (cap < 2ull * g->L) cap = 2ull * g->L;
+  }
+  if (cap < 2ull * g->L || (cap & (cap - 1))) {
+    g->err = "capacity must be a power of two >= 2L";
+    return GPMA_ERR_INVALID_ARG;
+  }
+  set_geometry(g, cap);
+  if ((st = alloc_store(g, cap, &g->key, &g->val, &g->cnt, &g->head, s))) return st;
+  GP_CHECK(g, cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->V + 1) * 8, s));
+  GP_CHECK(g, cudaMemsetAsync(g->row_offset, 0, ((uint64_t)g->V + 1) * 8, s));
+  if (E > g->tmax[g->h] && !cap_override) {
+    g->err = "initial graph exceeds the root bound";
+    return GPMA_ERR_INVALID_ARG;
+  }
+  // dense merged list (edges + guards) in the window scratch
+  GP_CHECK(g, ensure(g->b_wk, std::max<uint64_t>(E, 1) * 8, s));
+  GP_CHECK(g, ensure(g->b_wv, std::max<uint64_t>(E, 1) * 4, s));
+  uint64_t *wk = (uint64_t *)g->b_wk.p;
+  uint32_t *wv = (uint32_t *)g->b_wv.p;
+  if (m) {
+    // positions: edge with unique rank j (pos) and source u goes to j + u
+    int which_unused = 0;
+    (void)which_unused;
+    uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p;
+    // recompute from the dense list: keep = 1, pos = j
+    // (the dense list ek is sorted & unique; place directly)
+    GP_LAUNCH(g, k_unique_last, grid_for(m), TB, 0, s, ek, m, keep);  // all ones (unique)
+    scan_u32(g, keep, pos, m, s);
+    GP_LAUNCH(g, k_place_edges, grid_for(m), TB, 0, s, ek, ev, pos, keep, m, wk, wv);
+  }
+  GP_LAUNCH(g, k_place_guards, grid_for(g->V), TB, 0, s, nullptr, g->V, ek, m, wk, wv);
+  GP_CHECK(g, cudaGetLastError());
+  return build_from_sorted(g, wk, wv, E, s);
+}
+
+// ---- one GPMA+ round (level `lvl`), generic device-scale implementation
+struct LevelOut {
+  uint64_t q, nacc, p_new;
+};
+
+static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t *dirty_base,
+                              cudaStream_t s, bool resize_target, uint64_t new_cap, uint64_t *nk,
+                              uint32_t *nv, uint32_t *ncnt) {
+  const uint64_t p = a.p;
+  const uint64_t nleaves = g->cap / g->L;
+  const uint64_t wins_bound = std::min<uint64_t>(p, nleaves >> a.lvl);
+  const uint64_t wslots = (uint64_t)g->L << a.lvl;
+  const unsigned gp = grid_for(p);
+  GP_LAUNCH(g, k_lvl_flags, gp, TB, 0, s, a);
+  scan_u32(g, a.hf, a.widx, p, s);
+  GP_LAUNCH(g, k_lvl_first, gp, TB, 0, s, a);
+  if (a.lvl <= 4) GP_LAUNCH(g, k_lvl_count<1>, grid_for(p), TB, 0, s, a, g->cnt);
+  else if (a.lvl <= 11) GP_LAUNCH(g, k_lvl_count<32>, grid_for(p * 32), TB, 0, s, a, g->cnt);
+  else GP_LAUNCH(g, k_lvl_count<TB>, (unsigned)std::min<uint64_t>(p, MAX_RESIDENT_BLOCKS), TB, 0, s, a, g->cnt);
+  scan_u32(g, a.acc, a.aidx, p, s);
+  scan_u64(g, a.nw, a.woff, p, s);
+  GP_LAUNCH(g, k_lvl_alist, gp, TB, 0, s, a);
+  // scratch: sum of merged window sizes <= wins_bound * wslots (and <= cap + p)
+  uint64_t need = a.force ? g->cap + p : wins_bound * wslots;
+  GP_CHECK(g, ensure(g->b_wk, need * 8, s));
+  GP_CHECK(g, ensure(g->b_wv, need * 4, s));
+  a.wk = (uint64_t *)g->b_wk.p;
+  a.wv = (uint32_t *)g->b_wv.p;
+  if (a.lvl) {
+    uint64_t lb = wins_bound << a.lvl;
+    GP_CHECK(g, ensure(g->b_lpre, (lb + 1) * 8, s));
+    a.lpre = (uint64_t *)g->b_lpre.p;
+    GP_LAUNCH(g, k_lvl_leafcnt, grid_for(lb), TB, 0, s, a, g->cnt, lb);
+    scan_u64(g, a.lpre, a.lpre, lb, s);
+  }
+  uint64_t bslots = wins_bound * wslots;
+  uint64_t bslots_r = (bslots + 31) & ~31ull;
+  GP_LAUNCH(g, k_lvl_gather, grid_for(bslots_r), TB, 0, s, a, g->key, g->val, bslots_r);
+  if (a.op == GPMA_INSERT) GP_LAUNCH(g, k_lvl_place, gp, TB, 0, s, a, g->key, g->val);
+  if (!resize_target) {
+    GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots), TB, 0, s, a, g->key, g->val, g->cnt,
+              g->row_offset, bslots, (uint2 *)g->b_dirty.p, *dirty_base);
+  } else {
+    // the single root window, laid out over the whole new array
+    uint64_t N;
+    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, a.nw, 8, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaStreamSynchronize(s));
+    N = g->ctrl_h->sum;
+    uint64_t nl_new = new_cap / g->L;
+    GP_LAUNCH(g, k_layout_even, grid_for(new_cap), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
+              g->row_offset, g->L, nl_new);
+  }
+  GP_LAUNCH(g, k_lvl_keep, gp, TB, 0, s, a);
+  scan_u32(g, a.keep, a.kpos, p, s);
+  GP_LAUNCH(g, k_lvl_summary, 1, 1, 0, s, a, g->ctrl_d);
+  if (g->trace_on) {
+    // copy segment starts / offsets / flags of this level (debug only)
+    std::vector<uint32_t> wf(p + 1), ac(p + 1), pt(p), wi(p + 1);
+    GP_CHECK(g, cudaMemcpyAsync(wf.data(), a.wfirst, (p + 1) * 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaMemcpyAsync(ac.data(), a.acc, p * 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaMemcpyAsync(pt.data(), a.pt, p * 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaMemcpyAsync(wi.data(), a.widx, (p + 1) * 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaStreamSynchronize(s));
+    uint32_t q = wi[p];
+    for (uint32_t w = 0; w < q; ++w) {
+      uint64_t start = ((uint64_t)(pt[wf[w]] >> a.lvl) << a.lvl) * g->L;
+      g->trace.insert(g->trace.end(), {a.lvl, start, wf[w], ac[w]});
+    }
+    g->trace.insert(g->trace.end(), {a.lvl, KEY_NONE, wf[q], 2});
+  }
+  gpma_status st = read_ctrl(g, s);
+  if (st) return st;
+  out->q = g->ctrl_h->sum & 0xFFFFFFFFull;
+  out->nacc = g->ctrl_h->sum >> 32;
+  out->p_new = g->ctrl_h->sum2;
+  *dirty_base += out->nacc;
+  // compact the pending list into the other buffer
+  if (out->p_new && !resize_target) {
+    GP_LAUNCH(g, k_compact_pending, grid_for(p), TB, 0, s, a.keep, a.kpos, p, a.pk, a.pv, a.pt,
+              (uint64_t *)g->b_pk[cur ^ 1].p, (uint32_t *)g->b_pv[cur ^ 1].p,
+              (uint32_t *)g->b_pt[cur ^ 1].p);
+  }
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+static gpma_status level_buffers(gpma *g, uint64_t n, cudaStream_t s) {
+  size_t b4 = (n + 2) * 4, b8 = (n + 2) * 8;
+  GP_CHECK(g, ensure(g->b_hf, b4, s));
+  GP_CHECK(g, ensure(g->b_widx, b4, s));
+  GP_CHECK(g, ensure(g->b_wfirst, b4, s));
+  GP_CHECK(g, ensure(g->b_acc, b4, s));
+  GP_CHECK(g, ensure(g->b_aidx, b4, s));
+  GP_CHECK(g, ensure(g->b_alist, b4, s));
+  GP_CHECK(g, ensure(g->b_keep2, b4, s));
+  GP_CHECK(g, ensure(g->b_kpos, b4, s));
+  GP_CHECK(g, ensure(g->b_nw, b8, s));
+  GP_CHECK(g, ensure(g->b_woff, b8, s));
+  GP_CHECK(g, ensure(g->b_dirty, (n + 2) * sizeof(uint2), s));
+  for (int i = 0; i < 2; ++i) {
+    GP_CHECK(g, ensure(g->b_pk[i], b8, s));
+    GP_CHECK(g, ensure(g->b_pv[i], b4, s));
+    GP_CHECK(g, ensure(g->b_pt[i], b4, s));
+  }
+  return GPMA_OK;
+}
+
+static Lvl make_lvl(gpma *g, int cur, uint64_t p, uint32_t lvl, int op) {
+  Lvl a{};
+  a.pk = (const uint64_t *)g->b_pk[cur].p;
+  a.pv = (const uint32_t *)g->b_pv[cur].p;
+  a.pt = (const uint32_t *)g->b_pt[cur].p;
+  a.p = p;
+  a.lvl = lvl;
+  a.L = g->L;
+  a.hf = (uint32_t *)g->b_hf.p;
+  a.widx = (uint32_t *)g->b_widx.p;
+  a.wfirst = (uint32_t *)g->b_wfirst.p;
+  a.acc = (uint32_t *)g->b_acc.p;
+  a.aidx = (uint32_t *)g->b_aidx.p;
+  a.alist = (uint32_t *)g->b_alist.p;
+  a.keep = (uint32_t *)g->b_keep2.p;
+  a.kpos = (uint32_t *)g->b_kpos.p;
+  a.nw = (uint64_t *)g->b_nw.p;
+  a.woff = (uint64_t *)g->b_woff.p;
+  a.lpre = (uint64_t *)g->b_lpre.p;
+  a.tmin = lvl < g->tmin.size() ? g->tmin[lvl] : 0;
+  a.tmax = lvl < g->tmax.size() ? g->tmax[lvl] : 0;
+  a.op = op;
+  a.force = 0;
+  return a;
+}
+
+// Root resize (Alg. 4 l.16-17; R14): double until the live entries plus the pending
+// insertions fit max_h of the new capacity; halve (strict deletes) while below min_h
+// and cap > 2L.  Everything is laid out evenly over the new array.
+static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, uint64_t *dirty_base) {
+  gpma_status st;
+  uint64_t nl = g->cap / g->L;
+  if ((st = zero_ctrl(g, s))) return st;
+  GP_LAUNCH(g, k_sum_cnt, grid_for(nl), TB, 0, s, g->cnt, nl, g->ctrl_d);
+  if ((st = read_ctrl(g, s))) return st;
+  const uint64_t ntot = g->ctrl_h->sum;
+  const uint64_t N = op == GPMA_INSERT ? ntot + p : ntot - p;
+  uint64_t cap = g->cap;
+  std::vector<uint64_t> mn, mx;
+  if (op == GPMA_INSERT) {
+    for (;;) {
+      uint32_t hh = ilog2(cap / g->L);
+      level_bounds(g->L, hh, g->rho0, g->rhoh, g->tau0, g->tauh, mn, mx);
+      if (N <= mx[hh]) break;
+      cap *= 2;
+    }
+  } else {
+    for (;;) {
+      uint32_t hh = ilog2(cap / g->L);
+      level_bounds(g->L, hh, g->rho0, g->rhoh, g->tau0, g->tauh, mn, mx);
+      if (!(cap > 2ull * g->L && N < mn[hh])) break;
+      level_bounds(g->L, hh - 1, g->rho0, g->rhoh, g->tau0, g->tauh, mn, mx);
+      if (N > mx[hh - 1]) break;
+      cap /= 2;
+    }
+  }
+  uint64_t *nk = g->key;
+  uint32_t *nv = g->val, *ncnt = g->cnt;
+  uint64_t *nhead = g->head;
+  if (cap != g->cap) {
+    if ((st = alloc_store(g, cap, &nk, &nv, &ncnt, &nhead, s))) return st;
+  }
+  Lvl a = make_lvl(g, cur, p, g->h, op);
+  a.force = 1;
+  LevelOut lo{};
+  if ((st = level_step(g, a, cur, &lo, dirty_base, s, true, cap, nk, nv, ncnt))) return st;
+  if (cap != g->cap) {
+    cudaFreeAsync(g->key, s);
+    cudaFreeAsync(g->val, s);
+    cudaFreeAsync(g->cnt, s);
+    cudaFreeAsync(g->head, s);
+    g->key = nk;
+    g->val = nv;
+    g->cnt = ncnt;
+    g->head = nhead;
+    g->resizes++;
+    g->last.last_resized = 1;
+  }
+  set_geometry(g, cap);
+  g->last.last_slots_rewritten += cap;
+  g->last.last_windows_rewritten += 1;
+  return recompute_heads(g, s);
+}
+
+gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op,
+                         cudaStream_t s) {
+  gpma_status st;
+  g->last = gpma_stats_t{};
+  g->trace.clear();
+  if (n == 0) return GPMA_OK;
+  // stage (host or device input) -- sort_unique copies into its own buffers anyway
+  GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
+  GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
+  uint64_t *ik = (uint64_t *)g->b_stage[0].p;
+  uint32_t *iv = (uint32_t *)g->b_stage[1].p;
+  GP_CHECK(g, cudaMemcpyAsync(ik, keys, n * 8, cudaMemcpyDefault, s));
+  if (op == GPMA_INSERT) GP_CHECK(g, cudaMemcpyAsync(iv, vals, n * 4, cudaMemcpyDefault, s));
+  if ((st = validate(g, ik, iv, n, op == GPMA_INSERT, s))) return st;
+  int which;
+  uint64_t m;
+  if ((st = sort_unique(g, ik, op == GPMA_INSERT ? iv : nullptr, n, &m, false, &which, s))) return st;
+  const uint64_t *sk = (const uint64_t *)g->b_sk[which].p;
+  const uint32_t *sv = (const uint32_t *)g->b_sv[which].p;
+  GP_CHECK(g, ensure(g->b_keep, (n + 1) * 4, s));
+  GP_CHECK(g, ensure(g->b_pos, (n + 1) * 4, s));
+  GP_CHECK(g, ensure(g->b_tgt, (n + 1) * 4, s));
+  if ((st = level_buffers(g, n, s))) return st;
+  uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p, *tgt = (uint32_t *)g->b_tgt.p;
+  if ((st = zero_ctrl(g, s))) return st;
+  const uint64_t nl = g->cap / g->L;
+  GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt,
+            g->head, (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d);
+  scan_u32(g, keep, pos, n, s);
+  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, pos + n, 4, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->nunique, &g->ctrl_d->nunique, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  uint64_t p = (uint32_t)g->ctrl_h->sum2;
+  g->last.last_unique = g->ctrl_h->nunique;
+  g->last.last_pending = p;
+  if (p == 0) return GPMA_OK;
+  int cur = 0;
+  GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, tgt,
+            (uint64_t *)g->b_pk[0].p, (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p);
+  uint64_t dirty_base = 0;
+  uint32_t lvl = 0;
+  for (; lvl <= g->h && p > 0; ++lvl) {
+    Lvl a = make_lvl(g, cur, p, lvl, op);
+    LevelOut lo{};
+    if ((st = level_step(g, a, cur, &lo, &dirty_base, s, false, 0, nullptr, nullptr, nullptr))) return st;
+    g->last.last_slots_rewritten += lo.nacc * ((uint64_t)g->L << lvl);
+    g->last.last_windows_rewritten += lo.nacc;
+    g->last.last_top_level = lvl;
+    if (lo.p_new) cur ^= 1;
+    p = lo.p_new;
+  }
+  if (p > 0) {
+    g->last.last_top_level = g->h + 1;
+    if ((st = resize(g, cur, p, op, s, &dirty_base))) return st;
+    return GPMA_OK;
+  }
+  if (dirty_base) {
+    GP_LAUNCH(g, k_heads_dirty, grid_for(dirty_base * 32), TB, 0, s, g->key, g->head, g->L, nl,
+              (const uint2 *)g->b_dirty.p, dirty_base);
+  }
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+}  // namespace gp

@@ -1,0 +1,240 @@
+"""Thin ctypes binding of include/gpma.h (argument marshalling only).
+
+Every entry point forwards to the sm_100a library ``lib/libgpma.so``; there is no
+Python or CPU fallback -- importing this module on a machine without the built
+library raises, and the calls fail loudly without a CUDA device.
+
+Arrays may be torch tensors (CUDA or CPU; CPU tensors are passed as host pointers
+and staged by the library) or numpy arrays (host).  Keys are int64 tensors holding
+the u64 bits ``src << 32 | dst``; values int32 holding u32 bits.
+"""
+from __future__ import annotations
+
+import ctypes as C
+import os
+
+import numpy as np
+
+from .buildlib import LIB
+
+INSERT, DELETE = 0, 1
+DELETE_LAZY, DELETE_REBALANCE = 0, 1
+OK = 0
+STATUS = {0: "ok", 1: "invalid argument", 2: "vertex id out of range", 3: "reserved key or value",
+          4: "out of device memory", 5: "CUDA error", 6: "poisoned handle"}
+
+
+class GpmaError(RuntimeError):
+    def __init__(self, status: int, msg: str = ""):
+        super().__init__(f"gpma status {status} ({STATUS.get(status, '?')}): {msg}")
+        self.status = status
+
+
+class gpma_config(C.Structure):
+    _fields_ = [("struct_size", C.c_uint32), ("leaf_slots", C.c_uint32), ("initial_capacity", C.c_uint64),
+                ("rho_leaf_bp", C.c_uint16), ("rho_root_bp", C.c_uint16), ("tau_leaf_bp", C.c_uint16),
+                ("tau_root_bp", C.c_uint16), ("init_density_bp", C.c_uint16), ("reserved0", C.c_uint16),
+                ("delete_mode", C.c_uint32)]
+
+
+class gpma_stats_t(C.Structure):
+    _fields_ = [("num_vertices", C.c_uint32), ("leaf_slots", C.c_uint32), ("capacity", C.c_uint64),
+                ("height", C.c_uint32), ("delete_mode", C.c_uint32), ("live_edges", C.c_uint64),
+                ("tombstones", C.c_uint64), ("resizes", C.c_uint64), ("last_unique", C.c_uint64),
+                ("last_pending", C.c_uint64), ("last_slots_rewritten", C.c_uint64),
+                ("last_windows_rewritten", C.c_uint64), ("last_top_level", C.c_uint32),
+                ("last_resized", C.c_uint32)]
+
+
+_lib = None
+
+
+def lib() -> C.CDLL:
+    """Load libgpma.so (built by __graft_entry__.build()); raise if it is missing."""
+    global _lib
+    if _lib is None:
+        if not os.path.exists(LIB):
+            raise ImportError(f"libgpma.so not built at {LIB}: run __graft_entry__.build()")
+        L = C.CDLL(LIB)
+        P, u64, u32, i32, st = C.c_void_p, C.c_uint64, C.c_uint32, C.c_int, C.c_int
+        sig = {
+            "gpma_config_default": (None, [P]),
+            "gpma_create": (st, [u32, P, P, u64, P, P, P]),
+            "gpma_create_raw": (st, [u32, u64, u32, P, P, P, P, P]),
+            "gpma_destroy": (st, [P]),
+            "gpma_update_batch": (st, [P, P, P, u64, i32, P]),
+            "gpma_bfs": (st, [P, u32, P, P]),
+            "gpma_cc": (st, [P, P, P]),
+            "gpma_pagerank": (st, [P, P, i32, C.c_double, C.c_double, i32, P, P]),
+            "gpma_pagerank_f32": (st, [P, P, i32, C.c_float, C.c_float, i32, P, P]),
+            "gpma_export_csr": (st, [P, P, P, P, u64, P, P]),
+            "gpma_stats": (st, [P, P]),
+            "gpma_debug_dump": (st, [P, P, P, P, P, P, P]),
+            "gpma_debug_set_trace": (st, [P, i32]),
+            "gpma_debug_trace": (st, [P, P, u64, P]),
+            "gpma_kernel_launches": (u64, [P]),
+            "gpma_status_string": (C.c_char_p, [st]),
+            "gpma_last_error": (C.c_char_p, [P]),
+        }
+        for name, (res, args) in sig.items():
+            f = getattr(L, name)
+            f.restype, f.argtypes = res, args
+        _lib = L
+    return _lib
+
+
+EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destroy", "gpma_update_batch",
+           "gpma_bfs", "gpma_cc", "gpma_pagerank", "gpma_pagerank_f32", "gpma_export_csr", "gpma_stats",
+           "gpma_debug_dump", "gpma_debug_set_trace", "gpma_debug_trace", "gpma_kernel_launches",
+           "gpma_status_string", "gpma_last_error"]
+
+
+def _ptr(a):
+    """Raw pointer of a torch tensor / numpy array (None passes NULL)."""
+    if a is None:
+        return None
+    if hasattr(a, "data_ptr"):
+        if not a.is_contiguous():
+            raise ValueError("array must be contiguous")
+        return a.data_ptr() or None
+    if isinstance(a, np.ndarray):
+        if not a.flags["C_CONTIGUOUS"]:
+            raise ValueError("array must be contiguous")
+        return a.ctypes.data or None
+    raise TypeError(type(a))
+
+
+def _numel(a) -> int:
+    return int(a.numel()) if hasattr(a, "numel") else int(a.size)
+
+
+def _stream(stream):
+    if stream is None:
+        try:
+            import torch
+            if torch.cuda.is_available():
+                return torch.cuda.current_stream().cuda_stream or None
+        except Exception:
+            pass
+        return None
+    if isinstance(stream, int):
+        return stream or None
+    return stream.cuda_stream or None
+
+
+class Gpma:
+    """One GPMA+ store (one handle of the C ABI).  Method names follow gpma.h."""
+
+    def __init__(self, handle, num_vertices):
+        self._h = handle
+        self.V = num_vertices
+
+    # -- create / destroy -------------------------------------------------
+    @classmethod
+    def gpma_create(cls, num_vertices: int, init_keys=None, init_vals=None, *, leaf_slots: int = 0,
+                    initial_capacity: int = 0, delete_mode: int = DELETE_LAZY, thresholds_bp=None,
+                    init_density_bp: int = 6000, stream=None) -> "Gpma":
+        cfg = gpma_config()
+        lib().gpma_config_default(C.byref(cfg))
+        cfg.leaf_slots = leaf_slots
+        cfg.initial_capacity = initial_capacity
+        cfg.delete_mode = delete_mode
+        cfg.init_density_bp = init_density_bp
+        if thresholds_bp:
+            cfg.rho_leaf_bp, cfg.rho_root_bp, cfg.tau_leaf_bp, cfg.tau_root_bp = thresholds_bp
+        h = C.c_void_p()
+        n = 0 if init_keys is None else _numel(init_keys)
+        st = lib().gpma_create(num_vertices, _ptr(init_keys), _ptr(init_vals), n, C.byref(cfg),
+                               _stream(stream), C.byref(h))
+        if st != OK:
+            raise GpmaError(st, "gpma_create")
+        return cls(h, num_vertices)
+
+    @classmethod
+    def gpma_create_raw(cls, num_vertices: int, capacity: int, leaf_slots: int, keys, vals, *,
+                        delete_mode: int = DELETE_LAZY, stream=None) -> "Gpma":
+        cfg = gpma_config()
+        lib().gpma_config_default(C.byref(cfg))
+        cfg.delete_mode = delete_mode
+        h = C.c_void_p()
+        st = lib().gpma_create_raw(num_vertices, capacity, leaf_slots, _ptr(keys), _ptr(vals), C.byref(cfg),
+                                   _stream(stream), C.byref(h))
+        if st != OK:
+            raise GpmaError(st, "gpma_create_raw")
+        return cls(h, num_vertices)
+
+    def gpma_destroy(self):
+        if self._h:
+            lib().gpma_destroy(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.gpma_destroy()
+        except Exception:
+            pass
+
+    def _check(self, st, what):
+        if st != OK:
+            msg = lib().gpma_last_error(self._h) if self._h else b""
+            raise GpmaError(st, f"{what}: {msg.decode() if msg else ''}")
+
+    # -- update -----------------------------------------------------------
+    def gpma_update_batch(self, keys, vals=None, op: int = INSERT, stream=None, check: bool = True) -> int:
+        st = lib().gpma_update_batch(self._h, _ptr(keys), _ptr(vals), _numel(keys), op, _stream(stream))
+        if check:
+            self._check(st, "gpma_update_batch")
+        return st
+
+    def insert(self, keys, vals, stream=None):
+        return self.gpma_update_batch(keys, vals, INSERT, stream)
+
+    def delete(self, keys, stream=None):
+        return self.gpma_update_batch(keys, None, DELETE, stream)
+
+    # -- analytics --------------------------------------------------------
+    def gpma_bfs(self, root: int, levels, stream=None):
+        self._check(lib().gpma_bfs(self._h, root, _ptr(levels), _stream(stream)), "gpma_bfs")
+        return levels
+
+    def gpma_cc(self, labels, stream=None):
+        self._check(lib().gpma_cc(self._h, _ptr(labels), _stream(stream)), "gpma_cc")
+        return labels
+
+    def gpma_pagerank(self, rank, warm_start: bool = False, damping: float = 0.85, tol_l1: float = 1e-3,
+                      max_iter: int = 100, stream=None) -> int:
+        it = C.c_int(0)
+        f = lib().gpma_pagerank_f32 if str(getattr(rank, "dtype", "")).endswith("float32") else lib().gpma_pagerank
+        self._check(f(self._h, _ptr(rank), int(warm_start), damping, tol_l1, max_iter, C.byref(it),
+                      _stream(stream)), "gpma_pagerank")
+        return it.value
+
+    def gpma_export_csr(self, row_ptr=None, col=None, val=None, stream=None) -> int:
+        nnz = C.c_uint64(0)
+        cap = 0 if col is None else _numel(col)
+        self._check(lib().gpma_export_csr(self._h, _ptr(row_ptr), _ptr(col), _ptr(val), cap, C.byref(nnz),
+                                          _stream(stream)), "gpma_export_csr")
+        return nnz.value
+
+    # -- introspection ----------------------------------------------------
+    def gpma_stats(self) -> dict:
+        s = gpma_stats_t()
+        self._check(lib().gpma_stats(self._h, C.byref(s)), "gpma_stats")
+        return {f: getattr(s, f) for f, _ in s._fields_}
+
+    def gpma_debug_dump(self, keys=None, vals=None, row_offset=None, leaf_live=None, heads=None, stream=None):
+        self._check(lib().gpma_debug_dump(self._h, _ptr(keys), _ptr(vals), _ptr(row_offset), _ptr(leaf_live),
+                                          _ptr(heads), _stream(stream)), "gpma_debug_dump")
+
+    def gpma_debug_set_trace(self, enable: bool):
+        self._check(lib().gpma_debug_set_trace(self._h, int(enable)), "gpma_debug_set_trace")
+
+    def gpma_debug_trace(self):
+        n = C.c_uint64(0)
+        lib().gpma_debug_trace(self._h, None, 0, C.byref(n))
+        buf = np.zeros(4 * max(n.value, 1), np.uint64)
+        lib().gpma_debug_trace(self._h, buf.ctypes.data, n.value, C.byref(n))
+        return buf[: 4 * n.value].reshape(-1, 4)
+
+    def gpma_kernel_launches(self) -> int:
+        return int(lib().gpma_kernel_launches(self._h))

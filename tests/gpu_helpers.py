@@ -1,0 +1,109 @@
+"""Shared helpers for the GPU parity tests (compare the CUDA path with the oracle)."""
+from __future__ import annotations
+
+import numpy as np
+import torch
+
+import oracle as O
+
+KEY_NONE = np.uint64(0xFFFFFFFFFFFFFFFF)
+DEV = "cuda:0"
+
+
+def gpu_dump(g):
+    st = g.gpma_stats()
+    cap, L = st["capacity"], st["leaf_slots"]
+    nl = cap // L
+    k = torch.empty(cap, dtype=torch.int64, device=DEV)
+    v = torch.empty(cap, dtype=torch.int32, device=DEV)
+    ro = torch.empty(g.V + 1, dtype=torch.int64, device=DEV)
+    cnt = torch.empty(nl, dtype=torch.int32, device=DEV)
+    hd = torch.empty(nl, dtype=torch.int64, device=DEV)
+    g.gpma_debug_dump(k, v, ro, cnt, hd)
+    torch.cuda.synchronize()
+    return (k.cpu().numpy().view(np.uint64), v.cpu().numpy().view(np.uint32), ro.cpu().numpy().view(np.uint64),
+            cnt.cpu().numpy().view(np.uint32), hd.cpu().numpy().view(np.uint64), st)
+
+
+def expected_heads(keys, L):
+    """R9 locate index: head[l] = first key of the first non-empty leaf >= l (KEY_NONE if none)."""
+    first = keys.reshape(-1, L)[:, 0]
+    out = np.empty_like(first)
+    nxt = KEY_NONE
+    for l in range(first.size - 1, -1, -1):
+        if first[l] != KEY_NONE:
+            nxt = first[l]
+        out[l] = nxt
+    return out
+
+
+def expected_leaf_live(keys, vals, L):
+    occ = (keys != KEY_NONE) & (vals != np.uint32(0xFFFFFFFF))
+    return occ.reshape(-1, L).sum(axis=1).astype(np.uint32)
+
+
+def assert_same_layout(g, o: O.Oracle, guards=True, what=""):
+    gk, gv, gro, gcnt, ghd, st = gpu_dump(g)
+    ok, ov = o.dump()
+    assert gk.size == ok.size, f"{what}: capacity {gk.size} != oracle {ok.size}"
+    if not np.array_equal(gk, ok):
+        bad = np.nonzero(gk != ok)[0]
+        raise AssertionError(f"{what}: {bad.size} slot keys differ, first at {bad[:8]}: "
+                             f"gpu {gk[bad[:4]]} oracle {ok[bad[:4]]}")
+    assert np.array_equal(gv, ov), f"{what}: slot values differ at {np.nonzero(gv != ov)[0][:8]}"
+    if guards:
+        assert np.array_equal(gro, o.row_offset()), f"{what}: row offsets differ"
+    L = st["leaf_slots"]
+    assert np.array_equal(gcnt, expected_leaf_live(ok, ov, L)), f"{what}: leaf live counts differ"
+    assert np.array_equal(ghd, expected_heads(ok, L)), f"{what}: locate heads differ"
+    return st
+
+
+def gpu_export(g):
+    nnz = g.gpma_export_csr()
+    rp = torch.empty(g.V + 1, dtype=torch.int64, device=DEV)
+    col = torch.empty(max(nnz, 1), dtype=torch.int32, device=DEV)
+    val = torch.empty(max(nnz, 1), dtype=torch.int32, device=DEV)
+    g.gpma_export_csr(rp, col, val)
+    torch.cuda.synchronize()
+    return (rp.cpu().numpy().view(np.uint64), col.cpu().numpy().view(np.uint32)[:nnz],
+            val.cpu().numpy().view(np.uint32)[:nnz])
+
+
+def assert_same_csr(g, o, what=""):
+    grp, gcol, gval = gpu_export(g)
+    orp, ocol, oval = o.export_csr()
+    assert np.array_equal(grp, orp), f"{what}: row_ptr differs"
+    assert np.array_equal(gcol, ocol), f"{what}: col differs"
+    assert np.array_equal(gval, oval), f"{what}: val differs"
+    return orp, ocol
+
+
+def gpu_bfs(g, root):
+    lv = torch.empty(g.V, dtype=torch.int32, device=DEV)
+    g.gpma_bfs(root, lv)
+    return lv.cpu().numpy()
+
+
+def gpu_cc(g):
+    lab = torch.empty(g.V, dtype=torch.int32, device=DEV)
+    g.gpma_cc(lab)
+    return lab.cpu().numpy().view(np.uint32)
+
+
+def gpu_pr(g, x=None, tol=0.0, max_iter=20, dtype=torch.float64):
+    if x is None:
+        xt = torch.empty(g.V, dtype=dtype, device=DEV)
+        it = g.gpma_pagerank(xt, warm_start=False, tol_l1=tol, max_iter=max_iter)
+    else:
+        xt = torch.as_tensor(x, dtype=dtype).to(DEV).contiguous()
+        it = g.gpma_pagerank(xt, warm_start=True, tol_l1=tol, max_iter=max_iter)
+    return xt.cpu().numpy().astype(np.float64), it
+
+
+def keys_t(keys):
+    return torch.as_tensor(np.asarray(keys, dtype=np.uint64).view(np.int64)).to(DEV)
+
+
+def vals_t(vals):
+    return torch.as_tensor(np.asarray(vals, dtype=np.uint32).view(np.int32)).to(DEV)
