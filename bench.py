@@ -1,0 +1,444 @@
+#!/usr/bin/env python
+"""GPMA+ benchmark: sliding-window edge updates + post-update analytics on B200.
+
+One STEP = one pass of the whole hot path (every row) over one slide of
+BASELINE.json configs[2] (Graph500 RMAT scale-24, edge factor 16, 1M-edge batches):
+    DELETE(expired 2^20) -> INSERT(arrived 2^20) -> BFS(random root) -> CC
+    -> PageRank(warm start, L1 < 1e-3) -> export_csr
+all through the C ABI of libgpma.so (sm_100a kernels), inputs already resident in HBM.
+
+metric = edge updates/s = (#deleted + #inserted keys) / step time (whole job, all ranks).
+`e2e` repeats the step through the same C ABI with HOST (pinned) buffers: the slide's
+batches go H2D inside the call and every result (BFS levels, CC labels, PR vector,
+exported CSR) comes back D2H.  `roofline` reports the dominant kernel's algorithmic
+bytes per launch / its CUDA-event-timed launch duration, against MEASURED_PEAKS.json.
+`cpu_baseline` times the CPU oracle (oracle/, single thread) on one slide of the same
+workload.  `--impl reference` is the reference arm: the oracle timed as it stands.
+
+Launch (N>1): python -m torch.distributed.run --nproc-per-node N --master-addr 127.0.0.1 ...
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import numpy as np  # noqa: E402
+import torch  # noqa: E402
+
+from gpma_gen import CONFIGS, bfs_root, config_stream  # noqa: E402
+
+L2_BYTES = 126 * 1024 * 1024
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--impl", default="gpma", choices=["gpma", "reference"])
+    ap.add_argument("--config", type=int, default=2)
+    ap.add_argument("--batch", type=int, default=0, help="override the slide batch size")
+    ap.add_argument("--pr-tol", type=float, default=1e-3)
+    ap.add_argument("--e2e-steps", type=int, default=5)
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--cpu-sample-batch", type=int, default=0)
+    ap.add_argument("--ref-sample-batch", type=int, default=1 << 16)
+    ap.add_argument("--profile-all", action="store_true", help="print the per-kernel time table")
+    return ap.parse_args()
+
+
+def peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        with open(p) as f:
+            d = json.load(f)
+        return float(d["hbm_gbs"]), "measured"
+    return 6650.0, "fallback"
+
+
+# ------------------------------------------------------------------ clocks
+class Clocks:
+    FIELDS = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,"
+              "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+              "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.proc = None
+        self.path = os.path.join("/tmp", f"gpma_clocks_{os.getpid()}.csv")
+        try:
+            self.f = open(self.path, "w")
+            self.proc = subprocess.Popen(["nvidia-smi", "-i", str(index), f"--query-gpu={self.FIELDS}",
+                                          "--format=csv,noheader,nounits", "-lms", "200"],
+                                         stdout=self.f, stderr=subprocess.DEVNULL)
+        except Exception:
+            self.proc = None
+
+    def stop(self) -> dict:
+        if self.proc is None:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        time.sleep(0.25)
+        self.proc.terminate()
+        self.proc.wait()
+        self.f.close()
+        sm, mx, reasons = [], [], set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for line in open(self.path):
+            parts = [x.strip() for x in line.split(",")]
+            if len(parts) < 6:
+                continue
+            try:
+                sm.append(float(parts[0]))
+                mx.append(float(parts[1]))
+            except ValueError:
+                continue
+            for n, v in zip(names, parts[2:6]):
+                if v.lower().startswith("active"):
+                    reasons.add(n)
+        os.unlink(self.path)
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+# ------------------------------------------------------------------ algorithmic bytes
+def algo_bytes(kernel: str, cap: int, V: int, L: int, nnz: int, dtype_bytes: int = 8) -> int | None:
+    """Algorithmic bytes of ONE launch of the kernel."""
+    if kernel == "k_pr_push":      # read key+val of every slot, contrib once per vertex, y RMW once
+        return 12 * cap + dtype_bytes * V + 2 * dtype_bytes * V
+    if kernel == "k_cc_hook":      # read key+val of every slot, parent array read+write once
+        return 12 * cap + 8 * V
+    if kernel == "k_pr_outdeg":
+        return 12 * cap + 4 * V
+    if kernel == "k_exp_leafcount":
+        return 12 * cap + 8 * (cap // L)
+    if kernel == "k_exp_write":    # read slots + leaf bases, write col/val + row_ptr
+        return 12 * cap + 8 * (cap // L) + 8 * nnz + 8 * (V + 1)
+    return None
+
+
+# ------------------------------------------------------------------ GPMA arm
+def run_gpma(args, rank, world, lrank):
+    from paper_journals_pvldb_shalht17_b200 import Gpma
+    dev = torch.device("cuda", lrank)
+    torch.cuda.set_device(dev)
+    cfg = CONFIGS[args.config]
+    t0 = time.time()
+    sw = config_stream(args.config, device=dev)
+    if args.batch:
+        sw.batch = args.batch
+    B, V = sw.batch, cfg.V
+    need = args.warmup + 1 + args.steps + (0 if args.no_e2e else 2 + args.e2e_steps)
+    assert need <= sw.n_slides, f"stream has {sw.n_slides} slides, need {need}"
+    gen_s = time.time() - t0
+    s = torch.cuda.Stream(dev)
+    with torch.cuda.stream(s):
+        k0, v0 = sw.initial()
+        g = Gpma.gpma_create(V, k0.contiguous(), v0.contiguous(), stream=s)
+        x = torch.empty(V, dtype=torch.float64, device=dev)
+        levels = torch.empty(V, dtype=torch.int32, device=dev)
+        labels = torch.empty(V, dtype=torch.int32, device=dev)
+        nnz_cap = sw.window + B
+        rp = torch.empty(V + 1, dtype=torch.int64, device=dev)
+        col = torch.empty(nnz_cap, dtype=torch.int32, device=dev)
+        cv = torch.empty(nnz_cap, dtype=torch.int32, device=dev)
+        g.gpma_pagerank(x, warm_start=False, tol_l1=args.pr_tol, max_iter=100, stream=s)
+        st0 = g.gpma_stats()
+        evs = []
+        pr_iters = []
+
+        def step(i, bufs=None):
+            dk, ik, iv = sw.slide(i)
+            root = bfs_root(sw, cfg.seed, i)
+            e = [torch.cuda.Event(enable_timing=True) for _ in range(7)]
+            e[0].record(s)
+            if bufs is None:
+                g.gpma_update_batch(dk, None, 1, stream=s)
+                e[1].record(s)
+                g.gpma_update_batch(ik, iv, 0, stream=s)
+                e[2].record(s)
+                g.gpma_bfs(root, levels, stream=s)
+                e[3].record(s)
+                g.gpma_cc(labels, stream=s)
+                e[4].record(s)
+                pr_iters.append(g.gpma_pagerank(x, warm_start=True, tol_l1=args.pr_tol, max_iter=100, stream=s))
+                e[5].record(s)
+                g.gpma_export_csr(rp, col, cv, stream=s)
+                e[6].record(s)
+            else:
+                hdk, hik, hiv, hx, hlv, hlab, hrp, hcol, hcv = bufs
+                g.gpma_update_batch(hdk, None, 1, stream=s)
+                e[1].record(s)
+                g.gpma_update_batch(hik, hiv, 0, stream=s)
+                e[2].record(s)
+                g.gpma_bfs(root, hlv, stream=s)
+                e[3].record(s)
+                g.gpma_cc(hlab, stream=s)
+                e[4].record(s)
+                pr_iters.append(g.gpma_pagerank(hx, warm_start=True, tol_l1=args.pr_tol, max_iter=100, stream=s))
+                e[5].record(s)
+                g.gpma_export_csr(hrp, hcol, hcv, stream=s)
+                e[6].record(s)
+            evs.append(e)
+
+        i = 0
+        for _ in range(args.warmup):
+            step(i)
+            i += 1
+        torch.cuda.synchronize()
+        # find the dominant kernel on the last warm-up shape (one profiled step, not timed)
+        g.gpma_debug_profile("*")
+        step(i)
+        i += 1
+        prof_all = g.gpma_debug_profile_read()
+        st = g.gpma_stats()
+        cap, L = st["capacity"], st["leaf_slots"]
+        nnz = st["live_edges"]
+        cand = {k: v for k, v in prof_all.items() if algo_bytes(k, cap, V, L, nnz) is not None}
+        dom = max(cand, key=lambda k: cand[k][1]) if cand else "k_pr_push"
+        evs.clear()
+        pr_iters.clear()
+        g.gpma_debug_profile(dom)
+        launches0 = g.gpma_kernel_launches()
+        if world > 1:
+            torch.distributed.barrier()
+        torch.cuda.synchronize()
+        clk = Clocks(lrank)
+        t_start = torch.cuda.Event(enable_timing=True)
+        t_end = torch.cuda.Event(enable_timing=True)
+        t_start.record(s)
+        for _ in range(args.steps):
+            step(i)
+            i += 1
+        t_end.record(s)
+        torch.cuda.synchronize()
+        if world > 1:
+            torch.distributed.barrier()
+        clocks = clk.stop()
+        ms = t_start.elapsed_time(t_end)
+        launches = g.gpma_kernel_launches() - launches0
+        prof_dom = g.gpma_debug_profile_read().get(dom, (0, 0.0))
+        g.gpma_debug_profile(None)
+        phase = np.array([[e[j].elapsed_time(e[j + 1]) for j in range(6)] for e in evs])
+        phase_ms = phase.mean(axis=0).tolist()
+        iters_timed = list(pr_iters)
+        st = g.gpma_stats()
+        cap = st["capacity"]
+
+        # ---- e2e through the C ABI with pinned host buffers
+        e2e = None
+        if not args.no_e2e:
+            evs.clear()
+            pr_iters.clear()
+            hx = x.cpu().pin_memory()
+            hlv = torch.empty(V, dtype=torch.int32).pin_memory()
+            hlab = torch.empty(V, dtype=torch.int32).pin_memory()
+            hrp = torch.empty(V + 1, dtype=torch.int64).pin_memory()
+            hcol = torch.empty(nnz_cap, dtype=torch.int32).pin_memory()
+            hcv = torch.empty(nnz_cap, dtype=torch.int32).pin_memory()
+            batches = []
+            for j in range(args.e2e_steps + 1):
+                dk, ik, iv = sw.slide(i + j)
+                batches.append((dk.cpu().pin_memory(), ik.cpu().pin_memory(), iv.cpu().pin_memory()))
+            step(i, (*batches[0], hx, hlv, hlab, hrp, hcol, hcv))   # warm-up of the host path
+            i += 1
+            torch.cuda.synchronize()
+            evs.clear()
+            pr_iters.clear()
+            t0e = time.perf_counter()
+            e0 = torch.cuda.Event(enable_timing=True)
+            e1 = torch.cuda.Event(enable_timing=True)
+            e0.record(s)
+            for j in range(args.e2e_steps):
+                step(i, (*batches[j + 1], hx, hlv, hlab, hrp, hcol, hcv))
+                i += 1
+            e1.record(s)
+            torch.cuda.synchronize()
+            wall = time.perf_counter() - t0e
+            ms_e2e = max(e0.elapsed_time(e1), wall * 1e3)
+            nnz_e = g.gpma_stats()["live_edges"]
+            h2d = B * (8 + 8 + 4) + 8 * V
+            d2h = 4 * V + 4 * V + 8 * V + 8 * (V + 1) + 8 * nnz_e
+            e2e = {"value": 2 * B * args.e2e_steps * world / (ms_e2e / 1e3), "unit": "edge updates/s",
+                   "ms_per_step": ms_e2e / args.e2e_steps, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
+                   "pr_iters": pr_iters}
+
+    # ---- max over ranks
+    t = torch.tensor([ms], dtype=torch.float64, device=dev)
+    if world > 1:
+        torch.distributed.all_reduce(t, op=torch.distributed.ReduceOp.MAX)
+    ms_max = float(t.item())
+    if rank != 0:
+        return
+    hbm, peak_kind = peaks()
+    nnz = st["live_edges"]
+    ab = algo_bytes(dom, cap, V, st["leaf_slots"], nnz)
+    n_l, tot_ms = prof_dom
+    avg_ms = tot_ms / n_l if n_l else float("nan")
+    achieved = ab / (avg_ms / 1e3) / 1e9 if n_l else None
+    out = {
+        "metric": "edge updates/sec (sliding window, 1M-edge delete+insert batches) with BFS/CC/PR/export after each update",
+        "value": 2 * B * args.steps * world / (ms_max / 1e3),
+        "unit": "edge updates/s",
+        "n_gpus": world,
+        "steps": args.steps,
+        "warmup": args.warmup,
+        "ms_per_step": ms_max / args.steps,
+        "higher_is_better": True,
+        "scaling": "weak",
+        "vs_baseline": None,
+        "dtype": "u64 keys / f64 PageRank",
+        "data": "synthetic (counter-based RMAT stream, gpma_gen)",
+        "config": {"workload": f"configs[{args.config}] {cfg.name}", "V": V, "stream_edges": cfg.E,
+                   "window": sw.window, "batch": B, "capacity": cap, "leaf_slots": st["leaf_slots"],
+                   "delete_mode": "lazy", "pr_tol": args.pr_tol,
+                   "parallelism": "replicas" if world > 1 else "single",
+                   "l2": "no flush: 3.2 GB store (> 126 MB L2) is streamed every step; each step reads a fresh batch"},
+        "breakdown_ms": {"delete": phase_ms[0], "insert": phase_ms[1], "bfs": phase_ms[2], "cc": phase_ms[3],
+                         "pagerank": phase_ms[4], "export_csr": phase_ms[5]},
+        "update_only": {"value": 2 * B / ((phase_ms[0] + phase_ms[1]) / 1e3), "unit": "edge updates/s",
+                        "ms_per_slide": phase_ms[0] + phase_ms[1]},
+        "pr_iters": iters_timed,
+        "roofline": {"bound": "hbm", "kernel": dom, "achieved": achieved, "peak": hbm, "unit": "GB/s",
+                     "frac": (achieved / hbm) if achieved else None, "traffic": None,
+                     "algorithmic_bytes_per_launch": ab, "avg_launch_ms": avg_ms, "launches": n_l,
+                     "peak_kind": peak_kind},
+        "e2e": e2e,
+        "gpu_launches": launches,
+        "clocks": clocks,
+        "setup_s": {"generate": gen_s},
+    }
+    if args.profile_all:
+        out["kernel_table_warm_step"] = {k: {"launches": v[0], "ms": v[1]} for k, v in
+                                         sorted(prof_all.items(), key=lambda kv: -kv[1][1])}
+    if world == 1 and not args.no_cpu_baseline:
+        out["cpu_baseline"] = cpu_baseline(sw, cfg, args, 0)
+    print(json.dumps(out))
+
+
+# ------------------------------------------------------------------ oracle legs
+def _oracle_step(o, sw, cfg, i, b, x, pr_tol):
+    import oracle as O  # noqa: F401  (test infrastructure: cpu_baseline / reference arm only)
+    dk, ik, iv = sw.slide(i)
+    dk, ik, iv = dk[:b].cpu().numpy(), ik[:b].cpu().numpy(), iv[:b].cpu().numpy()
+    root = bfs_root(sw, cfg.seed, i)
+    t = {}
+    c0 = time.perf_counter()
+    o.delete(dk)
+    o.insert(ik, iv)
+    c1 = time.perf_counter()
+    rp, col, _ = o.export_csr()
+    c2 = time.perf_counter()
+    from oracle import bfs_csr, cc_csr, pagerank_csr
+    bfs_csr(o.V, rp, col, root)
+    c3 = time.perf_counter()
+    cc_csr(o.V, rp, col)
+    c4 = time.perf_counter()
+    x, it = pagerank_csr(o.V, rp, col, x=x, tol=pr_tol, max_iter=100)
+    c5 = time.perf_counter()
+    t = {"update": c1 - c0, "export_csr": c2 - c1, "bfs": c3 - c2, "cc": c4 - c3, "pagerank": c5 - c4,
+         "pr_iters": it}
+    return c5 - c0, x, t
+
+
+def _oracle_setup(sw, V):
+    import oracle as O
+    k0, v0 = sw.initial()
+    o = O.Oracle(V, k0.cpu().numpy(), v0.cpu().numpy())
+    rp, col, _ = o.export_csr()
+    x, _ = O.pagerank_csr(V, rp, col, tol=1e-3, max_iter=100)
+    return o, x
+
+
+def cpu_baseline(sw, cfg, args, first_slide):
+    """The oracle as it stands, single-threaded, on one slide of the same workload."""
+    b = args.cpu_sample_batch or sw.batch
+    t0 = time.perf_counter()
+    o, x = _oracle_setup(sw, cfg.V)
+    setup = time.perf_counter() - t0
+    dt, x, parts = _oracle_step(o, sw, cfg, first_slide, b, x, args.pr_tol)
+    return {"value": 2 * b / dt, "unit": "edge updates/s", "cores": 1, "kind": "oracle",
+            "sample": f"1 slide of configs[{args.config}] ({b} deletes + {b} inserts on the full "
+                      f"{sw.window}-edge window, then export+BFS+CC+PR), single thread",
+            "step_s": dt, "parts_s": parts, "setup_s": setup,
+            "host": _cpu_model(), "host_cores": os.cpu_count()}
+
+
+def _cpu_model():
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                return line.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
+def run_reference(args, rank, world):
+    """Reference arm: the CPU oracle as it stands (no reference code exists for this paper)."""
+    if rank != 0:
+        return
+    cfg = CONFIGS[args.config]
+    dev = "cuda" if torch.cuda.is_available() else "cpu"
+    sw = config_stream(args.config, device=dev)
+    sw.keys, sw.vals = sw.keys.cpu(), sw.vals.cpu()
+    b = min(args.ref_sample_batch, sw.batch)
+    o, x = _oracle_setup(sw, cfg.V)
+    i = 0
+    for _ in range(args.warmup):
+        _, x, _ = _oracle_step(o, sw, cfg, i, b, x, args.pr_tol)
+        i += 1
+    tot = 0.0
+    parts = []
+    for _ in range(args.steps):
+        dt, x, p = _oracle_step(o, sw, cfg, i, b, x, args.pr_tol)
+        tot += dt
+        parts.append(p)
+        i += 1
+    val = 2 * b * args.steps / tot
+    out = {
+        "impl": "reference",
+        "metric": "edge updates/sec (sliding window, 1M-edge delete+insert batches) with BFS/CC/PR/export after each update",
+        "value": val, "unit": "edge updates/s", "n_gpus": world, "steps": args.steps, "warmup": args.warmup,
+        "ms_per_step": tot / args.steps * 1e3, "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+        "dtype": "u64 keys / f64 PageRank", "data": "synthetic (counter-based RMAT stream, gpma_gen)",
+        "config": {"workload": f"configs[{args.config}] {cfg.name}", "V": cfg.V, "window": sw.window,
+                   "batch": sw.batch, "sample_batch": b},
+        "cpu_baseline": {"value": val, "unit": "edge updates/s", "cores": 1, "kind": "oracle",
+                         "sample": f"each step: {b} deletes + {b} inserts of one slide on the full window, "
+                                   f"then export+BFS+CC+PR, single thread"},
+        "e2e": {"value": val, "unit": "edge updates/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+        "parts_s_mean": {k: float(np.mean([p[k] for p in parts])) for k in parts[0]} if parts else {},
+    }
+    print(json.dumps(out))
+
+
+def main():
+    args = parse()
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    lrank = int(os.environ.get("LOCAL_RANK", "0"))
+    if world > 1:
+        backend = "nccl" if torch.cuda.is_available() else "gloo"
+        if torch.cuda.is_available():
+            torch.cuda.set_device(lrank)
+        torch.distributed.init_process_group(backend)
+    try:
+        if args.impl == "reference":
+            run_reference(args, rank, world)
+        else:
+            run_gpma(args, rank, world, lrank)
+    finally:
+        if world > 1:
+            torch.distributed.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -157,6 +157,15 @@ gpma_status gpma_debug_set_trace(gpma_t *g, int enable);
  * carries the final offset.  Returns the record count in *count; copies at most max. */
 gpma_status gpma_debug_trace(gpma_t *g, uint64_t *out4, uint64_t max, uint64_t *count);
 
+/* Kernel profiler (bench evidence, CUDA events on the call's stream around each launch):
+ * filter NULL/"" = off, "*" = every kernel, else one kernel name (e.g. "k_pr_push").
+ * Setting the filter clears the records. */
+gpma_status gpma_debug_profile(gpma_t *g, const char *kernel_filter);
+/* Synchronises the stream of the recorded launches and writes one line per kernel name,
+ * "name<TAB>launches<TAB>total_ms\n", into buf (NUL-terminated, truncated to buflen);
+ * clears the records. */
+gpma_status gpma_debug_profile_read(gpma_t *g, char *buf, size_t buflen);
+
 /* Number of kernels this handle has launched since create (bench evidence). */
 uint64_t gpma_kernel_launches(const gpma_t *g);
 

@@ -4,7 +4,9 @@
 #include <cuda_runtime.h>
 #include <string.h>
 
+#include <map>
 #include <new>
+#include <string>
 
 #include "gpma_internal.cuh"
 
@@ -124,6 +126,7 @@ void free_handle(gpma *g) {
   if (g->head) cudaFreeAsync(g->head, s);
   if (g->row_offset) cudaFreeAsync(g->row_offset, s);
   cudaStreamSynchronize(s);
+  for (cudaEvent_t e : g->ev_pool) cudaEventDestroy(e);
   if (g->ctrl_d) cudaFree(g->ctrl_d);
   if (g->ctrl_h) cudaFreeHost(g->ctrl_h);
   cudaGetLastError();
@@ -367,6 +370,43 @@ gpma_status gpma_debug_trace(gpma_t *g, uint64_t *out4, uint64_t max, uint64_t *
   uint64_t n = g->trace.size() / 4;
   *count = n;
   if (out4) memcpy(out4, g->trace.data(), (n < max ? n : max) * 4 * sizeof(uint64_t));
+  return GPMA_OK;
+}
+
+gpma_status gpma_debug_profile(gpma_t *g, const char *kernel_filter) {
+  if (!g) return GPMA_ERR_INVALID_ARG;
+  g->prof_filter = kernel_filter ? kernel_filter : "";
+  g->prof_recs.clear();
+  g->ev_used = 0;
+  return GPMA_OK;
+}
+
+gpma_status gpma_debug_profile_read(gpma_t *g, char *buf, size_t buflen) {
+  if (!g || !buf || !buflen) return GPMA_ERR_INVALID_ARG;
+  if (cudaError_t e = cudaDeviceSynchronize()) return gp::cuda_fail(g, e, "profile_read");
+  std::map<std::string, std::pair<uint64_t, double>> agg;
+  for (auto &r : g->prof_recs) {
+    float ms = 0.f;
+    cudaEventElapsedTime(&ms, g->ev_pool[r.e0], g->ev_pool[r.e1]);
+    std::string nm(r.name);
+    size_t lt = nm.find('<');
+    if (lt != std::string::npos) nm = nm.substr(0, lt);
+    auto &a = agg[nm];
+    a.first += 1;
+    a.second += ms;
+  }
+  std::string out;
+  char line[256];
+  for (auto &kv : agg) {
+    snprintf(line, sizeof line, "%s\t%llu\t%.6f\n", kv.first.c_str(), (unsigned long long)kv.second.first,
+             kv.second.second);
+    out += line;
+  }
+  size_t n = out.size() < buflen - 1 ? out.size() : buflen - 1;
+  memcpy(buf, out.data(), n);
+  buf[n] = 0;
+  g->prof_recs.clear();
+  g->ev_used = 0;
   return GPMA_OK;
 }
 

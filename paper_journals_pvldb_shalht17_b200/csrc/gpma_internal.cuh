@@ -85,15 +85,27 @@ struct gpma {
   bool trace_on = false;
   std::vector<uint64_t> trace;    // (level, start, offset, flag) x4
   cudaStream_t st = nullptr;
+
+  // kernel-level CUDA-event profiler (bench evidence; off by default)
+  std::string prof_filter;        // "" = off, "*" = every kernel, else exact kernel name
+  std::vector<cudaEvent_t> ev_pool;
+  size_t ev_used = 0;
+  struct ProfRec { const char *name; size_t e0, e1; };
+  std::vector<ProfRec> prof_recs;
 };
 
 // ---------------------------------------------------------------- helpers (host)
 namespace gp {
 
+bool prof_begin(gpma *g, const char *name, cudaStream_t s);
+void prof_end(gpma *g, cudaStream_t s);
+
 #define GP_LAUNCH(g, kernel, grid, block, smem, stream, ...)                 \
   do {                                                                       \
+    bool prof_ = !(g)->prof_filter.empty() && gp::prof_begin((g), #kernel, (stream)); \
     kernel<<<(grid), (block), (smem), (stream)>>>(__VA_ARGS__);              \
     (g)->launches++;                                                         \
+    if (prof_) gp::prof_end((g), (stream));                                  \
   } while (0)
 
 inline unsigned grid_for(uint64_t n, int block = 256, int max_blocks = MAX_RESIDENT_BLOCKS) {

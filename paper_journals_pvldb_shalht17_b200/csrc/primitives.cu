@@ -6,6 +6,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cstring>
 
 #include "gpma_internal.cuh"
 
@@ -33,6 +34,31 @@ void release(DevBuf &b, cudaStream_t s) {
   b.p = nullptr;
   b.bytes = 0;
 }
+
+// ------------------------------------------------------------------ kernel profiler
+static size_t take_event(gpma *g) {
+  if (g->ev_used == g->ev_pool.size()) {
+    cudaEvent_t e;
+    cudaEventCreate(&e);
+    g->ev_pool.push_back(e);
+  }
+  return g->ev_used++;
+}
+
+bool prof_begin(gpma *g, const char *name, cudaStream_t s) {
+  if (g->prof_filter != "*") {
+    // exact match on the kernel name without template arguments
+    const char *lt = strchr(name, '<');
+    size_t n = lt ? (size_t)(lt - name) : strlen(name);
+    if (g->prof_filter.size() != n || strncmp(g->prof_filter.c_str(), name, n) != 0) return false;
+  }
+  size_t e0 = take_event(g), e1 = take_event(g);
+  cudaEventRecord(g->ev_pool[e0], s);
+  g->prof_recs.push_back({name, e0, e1});
+  return true;
+}
+
+void prof_end(gpma *g, cudaStream_t s) { cudaEventRecord(g->ev_pool[g->prof_recs.back().e1], s); }
 
 gpma_status cuda_fail(gpma *g, cudaError_t e, const char *where) {
   if (e == cudaErrorMemoryAllocation) {

@@ -73,6 +73,8 @@ def lib() -> C.CDLL:
             "gpma_debug_set_trace": (st, [P, i32]),
             "gpma_debug_trace": (st, [P, P, u64, P]),
             "gpma_kernel_launches": (u64, [P]),
+            "gpma_debug_profile": (st, [P, C.c_char_p]),
+            "gpma_debug_profile_read": (st, [P, C.c_char_p, C.c_size_t]),
             "gpma_status_string": (C.c_char_p, [st]),
             "gpma_last_error": (C.c_char_p, [P]),
         }
@@ -86,6 +88,7 @@ def lib() -> C.CDLL:
 EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destroy", "gpma_update_batch",
            "gpma_bfs", "gpma_cc", "gpma_pagerank", "gpma_pagerank_f32", "gpma_export_csr", "gpma_stats",
            "gpma_debug_dump", "gpma_debug_set_trace", "gpma_debug_trace", "gpma_kernel_launches",
+           "gpma_debug_profile", "gpma_debug_profile_read",
            "gpma_status_string", "gpma_last_error"]
 
 
@@ -235,6 +238,19 @@ class Gpma:
         buf = np.zeros(4 * max(n.value, 1), np.uint64)
         lib().gpma_debug_trace(self._h, buf.ctypes.data, n.value, C.byref(n))
         return buf[: 4 * n.value].reshape(-1, 4)
+
+    def gpma_debug_profile(self, kernel_filter: str | None):
+        self._check(lib().gpma_debug_profile(self._h, kernel_filter.encode() if kernel_filter else None),
+                    "gpma_debug_profile")
+
+    def gpma_debug_profile_read(self) -> dict:
+        buf = C.create_string_buffer(1 << 16)
+        self._check(lib().gpma_debug_profile_read(self._h, buf, len(buf)), "gpma_debug_profile_read")
+        out = {}
+        for line in buf.value.decode().splitlines():
+            name, n, ms = line.split("\t")
+            out[name] = (int(n), float(ms))
+        return out
 
     def gpma_kernel_launches(self) -> int:
         return int(lib().gpma_kernel_launches(self._h))
