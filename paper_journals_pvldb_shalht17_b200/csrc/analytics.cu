@@ -2,16 +2,28 @@
 //
 // "CSR on GPMA" (Fig. 5): row u occupies slots [row_offset[u], row_offset[u+1]);
 // a slot holds an edge iff it is occupied, not a guard and not a tombstone -- the
-// IsEntryExist test of Alg. 2 l.10 / Alg. 3 l.4.
-//   BFS  (Table 1: Merrill et al. [37]): level-synchronous top-down frontier expansion,
-//        one warp per frontier row (Neighbour Gathering, Alg. 3), visited checks by CAS.
-//   CC   (Table 1: Soman et al. [43]): edge-centric hooking of roots (larger id under
-//        smaller) with CAS + path halving, then full pointer jumping -> min-id labels.
-//   PR   (Table 1: CUSP SpMV [2]): push SpMV over the live slots.
-//   export: CSR compaction via per-leaf edge counts + scan.
+// IsEntryExist test of Alg. 2 l.10 / Alg. 3 l.4.  Sweeps read the key array
+// and the per-leaf tombstone mask (8.25 B/slot) instead of key + value (12 B/slot); keys are
+// loaded with streaming (evict-first) hints so the random-access vertex arrays keep L2.
+//
+//   BFS  (Table 1: Merrill et al. [37]): level-synchronous top-down BFS.  A level's frontier
+//        is rebuilt from levels[] (bitmap + list, no atomics on the critical path); small
+//        frontiers expand their rows load-balanced over slots (Neighbour Gathering, Alg. 3);
+//        large ones sweep only the leaves whose source range meets the frontier.  Discovery
+//        is a plain store of the depth (every racing writer stores the same value).
+//   CC   (Table 1: Soman et al. [43]): hooking of roots (larger id under smaller) with CAS
+//        and path halving; a sampled first round (first edge of every (source, leaf) run),
+//        full compression, then a full pass that skips edges whose endpoints already share
+//        a parent.  Roots are component minima -> canonical min-id labels (R19).
+//   PR   (Table 1: CUSP SpMV [2]): push SpMV over the live slots with the
+//        store-maintained out-degrees; x' / error / dangling / next contribution fused.  The
+//        fp64 path accumulates y in exact 64-bit fixed point (2^-62 units; y <= total rank
+//        mass <= 1) with integer REDs: order-independent and within 2^-63 per term.
+//   export: per-leaf edge counts (leaf live counts minus guards), one scan, one sweep.
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cstring>
 
 #include "gpma_internal.cuh"
 
@@ -19,68 +31,264 @@ namespace gp {
 
 constexpr int TA = 256;
 
-__device__ __forceinline__ bool edge_at(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val,
-                                        uint64_t s, uint64_t *k) {
-  uint64_t x = key[s];
+// ------------------------------------------------------------------ slot access
+struct Slot4 {
+  uint64_t k[4];
+  uint32_t tb;   // tombstone bits of the four slots
+};
+
+// four consecutive slots (s4 % 4 == 0; L >= 4 so they share a leaf)
+__device__ __forceinline__ void load4(const uint64_t *__restrict__ key, const uint32_t *__restrict__ tmask,
+                                      uint32_t L, uint64_t s4, Slot4 &o) {
+  ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(key + s4));
+  ulonglong2 b = __ldcs(reinterpret_cast<const ulonglong2 *>(key + s4 + 2));
+  o.k[0] = a.x; o.k[1] = a.y; o.k[2] = b.x; o.k[3] = b.y;
+  o.tb = (__ldg(tmask + s4 / L) >> (uint32_t)(s4 % L)) & 0xFu;
+}
+
+__device__ __forceinline__ bool live_key(uint64_t k) { return k != KEY_NONE && (uint32_t)k != COL_GUARD; }
+__device__ __forceinline__ bool edge4(const Slot4 &o, int j) { return live_key(o.k[j]) && !((o.tb >> j) & 1u); }
+
+__device__ __forceinline__ bool edge_at(const uint64_t *__restrict__ key, const uint32_t *__restrict__ tmask,
+                                        uint32_t L, uint64_t s, uint64_t *k) {
+  uint64_t x = __ldcs(key + s);
   *k = x;
-  return x != KEY_NONE && (uint32_t)x != COL_GUARD && val[s] != VAL_TOMB;
+  if (!live_key(x)) return false;
+  return !((__ldg(tmask + s / L) >> (uint32_t)(s % L)) & 1u);
+}
+
+__device__ __forceinline__ uint32_t upper_bound_u64(const uint64_t *__restrict__ a, uint32_t lo, uint32_t hi,
+                                                    uint64_t x) {
+  while (lo < hi) {
+    uint32_t mid = (lo + hi) >> 1;
+    if (a[mid] <= x) lo = mid + 1;
+    else hi = mid;
+  }
+  return lo;
+}
+
+// ------------------------------------------------------------------ out-degrees
+// out-degree of each row = live edges in it.  Per thread: runs of equal source over its 4
+// slots; the thread's first run is aggregated across the warp (hub rows span many lanes).
+__global__ void __launch_bounds__(TA) k_deg_count(const uint64_t *__restrict__ key,
+                                                  const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
+                                                  uint32_t *deg) {
+  const int lane = threadIdx.x & 31;
+  const uint64_t n4 = cap / 4, n4r = (n4 + 31) & ~31ull;
+  for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4r;
+       t += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t first_src = 0xFFFFFFFFu, first_cnt = 0, cur = 0xFFFFFFFFu, c = 0;
+    bool in_first = true;
+    if (t < n4) {
+      Slot4 sl;
+      load4(key, tmask, L, t * 4, sl);
+#pragma unroll
+      for (int j = 0; j < 4; ++j) {
+        if (!edge4(sl, j)) continue;
+        uint32_t u = (uint32_t)(sl.k[j] >> 32);
+        if (u == cur) { ++c; continue; }
+        if (c) {
+          if (in_first) { first_src = cur; first_cnt = c; in_first = false; }
+          else atomicAdd(&deg[cur], c);
+        }
+        cur = u;
+        c = 1;
+      }
+      if (c) {
+        if (in_first) { first_src = cur; first_cnt = c; }
+        else atomicAdd(&deg[cur], c);
+      }
+    }
+    uint32_t peers = __match_any_sync(0xffffffffu, first_src);
+    uint32_t sum = __reduce_add_sync(peers, first_cnt);
+    if (first_src != 0xFFFFFFFFu && (__ffs(peers) - 1) == lane) atomicAdd(&deg[first_src], sum);
+  }
+}
+
+gpma_status recompute_degrees(gpma *g, cudaStream_t s) {
+  GP_CHECK(g, cudaMemsetAsync(g->deg, 0, (uint64_t)g->V * 4, s));
+  GP_LAUNCH(g, k_deg_count, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, g->deg);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
 }
 
 // ------------------------------------------------------------------ BFS
-__global__ void k_bfs_init(int32_t *levels, uint32_t V, uint32_t root, uint32_t *frontier) {
+__global__ void k_bfs_init(int32_t *levels, uint32_t V, uint32_t root) {
   for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
        v += (uint64_t)gridDim.x * blockDim.x)
     levels[v] = (v == root) ? 0 : -1;
-  if (blockIdx.x == 0 && threadIdx.x == 0) frontier[0] = root;
 }
 
-__global__ void k_bfs_expand(const uint32_t *__restrict__ frontier, uint32_t fsize,
-                             const uint64_t *__restrict__ row_offset, const uint64_t *__restrict__ key,
-                             const uint32_t *__restrict__ val, int32_t *levels, int32_t depth,
-                             uint32_t *__restrict__ next, uint32_t *next_count) {
+// frontier of depth d: bitmap words written whole by one lane per 32 vertices; size into *F
+// (one atomic per CTA)
+__global__ void k_bfs_frontier(const int32_t *__restrict__ levels, uint32_t V, int32_t d,
+                               uint32_t *__restrict__ bm, uint32_t *F) {
+  __shared__ uint32_t cnt;
+  if (threadIdx.x == 0) cnt = 0;
+  __syncthreads();
   const int lane = threadIdx.x & 31;
-  const uint32_t lt = (1u << lane) - 1u;
-  const uint64_t warps = (uint64_t)gridDim.x * (blockDim.x / 32);
-  for (uint64_t i = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32; i < fsize; i += warps) {
-    uint32_t u = frontier[i];
-    uint64_t a = row_offset[u], b = row_offset[u + 1];
-    for (uint64_t s0 = a; s0 < b; s0 += 32) {
-      uint64_t s = s0 + lane;
-      bool disc = false;
-      uint32_t v = 0;
-      uint64_t k;
-      if (s < b && edge_at(key, val, s, &k)) {
-        v = (uint32_t)k;
-        if (levels[v] == -1) disc = atomicCAS(&levels[v], -1, depth) == -1;
-      }
-      uint32_t bal = __ballot_sync(0xffffffffu, disc);
-      if (bal) {
-        uint32_t base = 0;
-        if (lane == 0) base = atomicAdd(next_count, __popc(bal));
-        base = __shfl_sync(0xffffffffu, base, 0);
-        if (disc) next[base + __popc(bal & lt)] = v;
-      }
+  const uint64_t Vr = ((uint64_t)V + 31) & ~31ull;
+  uint32_t mine = 0;
+  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < Vr;
+       v += (uint64_t)gridDim.x * blockDim.x) {
+    bool in = v < V && levels[v] == d;
+    uint32_t bal = __ballot_sync(0xffffffffu, in);
+    if (lane == 0) {
+      bm[v >> 5] = bal;
+      mine += __popc(bal);
+    }
+  }
+  if (lane == 0 && mine) atomicAdd(&cnt, mine);
+  __syncthreads();
+  if (threadIdx.x == 0 && cnt) atomicAdd(F, cnt);
+}
+
+// frontier list from the bitmap (sparse levels only: few set bits)
+__global__ void k_bfs_list(const uint32_t *__restrict__ bm, uint32_t nwords, uint32_t *__restrict__ list,
+                           uint32_t *n) {
+  for (uint64_t w = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; w < nwords;
+       w += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t b = bm[w];
+    if (!b) continue;
+    uint32_t base = atomicAdd(n, (uint32_t)__popc(b));
+    while (b) {
+      int i = __ffs(b) - 1;
+      b &= b - 1;
+      list[base++] = (uint32_t)(w * 32 + i);
     }
   }
 }
 
+__global__ void k_bfs_rowlen(const uint32_t *__restrict__ frontier, uint32_t F,
+                             const uint64_t *__restrict__ row_offset, uint64_t *__restrict__ len) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < F;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t u = frontier[i];
+    len[i] = row_offset[u + 1] - row_offset[u];
+  }
+}
+
+// Sparse levels -- Neighbour Gathering over the concatenated frontier rows (Alg. 3),
+// load-balanced: warp w owns the contiguous slot range [w*C, (w+1)*C) of the concatenation,
+// binary-searches its first row once, then walks forward 32 slots at a time.
+__global__ void __launch_bounds__(TA) k_bfs_expand(const uint32_t *__restrict__ frontier, uint32_t F,
+                                                   const uint64_t *__restrict__ off,
+                                                   const uint64_t *__restrict__ row_offset,
+                                                   const uint64_t *__restrict__ key,
+                                                   const uint32_t *__restrict__ tmask, uint32_t L,
+                                                   int32_t *levels, int32_t depth) {
+  const int lane = threadIdx.x & 31;
+  const uint64_t total = off[F];
+  const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  const uint64_t w = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32;
+  const uint64_t chunk = ((total + nwarps - 1) / nwarps + 31) & ~31ull;
+  const uint64_t beg = w * chunk, end = min(beg + chunk, total);
+  if (beg >= end) return;
+  uint32_t i0 = 0;
+  if (lane == 0) i0 = upper_bound_u64(off, 0, F + 1, beg) - 1;
+  i0 = __shfl_sync(0xffffffffu, i0, 0);
+  for (uint64_t base = beg; base < end; base += 32) {
+    const uint64_t gi = base + lane;
+    uint32_t i = i0;
+    if (gi < end) {
+      while (off[i + 1] <= gi) ++i;
+      uint32_t u = frontier[i];
+      uint64_t s = row_offset[u] + (gi - off[i]);
+      uint64_t k;
+      if (edge_at(key, tmask, L, s, &k)) {
+        uint32_t v = (uint32_t)k;
+        if (levels[v] == -1) levels[v] = depth;
+      }
+    }
+    i0 = __shfl_sync(0xffffffffu, i, 31);
+  }
+}
+
+// A leaf is active when its source range holds a frontier vertex.  The range comes from the
+// locate heads (every vertex has a guard, so a leaf spans at most L sources).
+__global__ void k_bfs_leaf_active(const uint64_t *__restrict__ head, uint64_t nleaves, uint32_t V,
+                                  const uint32_t *__restrict__ bm, uint32_t *__restrict__ act) {
+  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
+       l += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t h0 = head[l], h1 = l + 1 < nleaves ? head[l + 1] : KEY_NONE;
+    uint32_t ua = h0 == KEY_NONE ? V : (uint32_t)(h0 >> 32);
+    uint32_t ub = h1 == KEY_NONE ? V - 1 : (uint32_t)(h1 >> 32);
+    uint32_t a = 0;
+    for (uint32_t u = ua; u <= ub && u < V; ++u)
+      if ((__ldg(bm + (u >> 5)) >> (u & 31)) & 1u) { a = 1; break; }
+    act[l] = a;
+  }
+}
+
+__global__ void k_bfs_leaf_list(const uint32_t *__restrict__ act, const uint32_t *__restrict__ apos,
+                                uint64_t nleaves, uint32_t *__restrict__ alist) {
+  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
+       l += (uint64_t)gridDim.x * blockDim.x)
+    if (act[l]) alist[apos[l]] = (uint32_t)l;
+}
+
+// Dense levels: sweep the active leaves, two groups of 4 slots per thread, expanding the
+// edges whose source is in the frontier bitmap.
+__global__ void __launch_bounds__(TA) k_bfs_sweep(const uint64_t *__restrict__ key,
+                                                  const uint32_t *__restrict__ tmask, uint32_t L,
+                                                  const uint32_t *__restrict__ alist,
+                                                  const uint32_t *__restrict__ nact_p,
+                                                  const uint32_t *__restrict__ bm, int32_t *levels,
+                                                  int32_t depth) {
+  const uint32_t tpl = L / 4;
+  const uint64_t n4 = (uint64_t)(*nact_p) * tpl;
+  for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4;
+       t += (uint64_t)gridDim.x * blockDim.x) {
+    Slot4 sl;
+    load4(key, tmask, L, (uint64_t)alist[t / tpl] * L + (t % tpl) * 4, sl);
+#pragma unroll
+    for (int j = 0; j < 4; ++j) {
+      if (!edge4(sl, j)) continue;
+      uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
+      if (!((__ldg(bm + (u >> 5)) >> (u & 31)) & 1u)) continue;
+      if (levels[v] == -1) levels[v] = depth;
+    }
+  }
+}
+
+constexpr uint32_t BFS_SPARSE_F = 4096;   // frontiers up to this size use row expansion
+
 gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
-  GP_CHECK(g, ensure(g->b_misc, ((uint64_t)g->V + 1) * 4, s));
-  GP_CHECK(g, ensure(g->b_misc2, ((uint64_t)g->V + 1) * 4, s));
-  uint32_t *fa = (uint32_t *)g->b_misc.p, *fb = (uint32_t *)g->b_misc2.p;
-  uint32_t *cnt_d = &reinterpret_cast<uint32_t *>(&g->ctrl_d->sum)[0];
-  GP_LAUNCH(g, k_bfs_init, grid_for(g->V), TA, 0, s, levels, g->V, root, fa);
-  uint32_t fsize = 1;
-  int32_t depth = 0;
-  while (fsize) {
-    ++depth;
-    GP_CHECK(g, cudaMemsetAsync(cnt_d, 0, 4, s));
-    GP_LAUNCH(g, k_bfs_expand, grid_for((uint64_t)fsize * 32), TA, 0, s, fa, fsize, g->row_offset,
-              g->key, g->val, levels, depth, fb, cnt_d);
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, cnt_d, 4, cudaMemcpyDeviceToHost, s));
+  const uint64_t V = g->V, nl = g->cap / g->L;
+  GP_CHECK(g, ensure(g->b_an[0], (V + 1) * 4, s));
+  GP_CHECK(g, ensure(g->b_an[2], (std::max<uint64_t>(V, nl) + 2) * 8, s));
+  GP_CHECK(g, ensure(g->b_an[3], (V / 32 + 2) * 4, s));
+  GP_CHECK(g, ensure(g->b_misc, (nl + 2) * 4, s));
+  uint32_t *list = (uint32_t *)g->b_an[0].p;
+  uint64_t *off = (uint64_t *)g->b_an[2].p;
+  uint32_t *act = (uint32_t *)g->b_an[2].p;          // shares off's buffer: never both in a level
+  uint32_t *apos = act + nl + 1;
+  uint32_t *alist = (uint32_t *)g->b_misc.p;
+  uint32_t *bm = (uint32_t *)g->b_an[3].p;
+  uint32_t *F_d = reinterpret_cast<uint32_t *>(&g->ctrl_d->sum);
+  const uint32_t *tmask = tmask_of(g);
+  GP_LAUNCH(g, k_bfs_init, grid_for(V), TA, 0, s, levels, (uint32_t)V, root);
+  for (int32_t depth = 1;; ++depth) {
+    GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
+    GP_LAUNCH(g, k_bfs_frontier, grid_for(V), TA, 0, s, levels, (uint32_t)V, depth - 1, bm, F_d);
+    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
-    fsize = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
-    std::swap(fa, fb);
+    const uint32_t F = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
+    if (!F) break;
+    if (F <= BFS_SPARSE_F) {
+      GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
+      GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, F_d);
+      GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, off);
+      scan_u64(g, off, off, F, s);
+      GP_LAUNCH(g, k_bfs_expand, MAX_RESIDENT_BLOCKS, TA, 0, s, list, F, off, g->row_offset, g->key, tmask,
+                g->L, levels, depth);
+    } else {
+      GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, act);
+      scan_u32(g, act, apos, nl, s);
+      GP_LAUNCH(g, k_bfs_leaf_list, grid_for(nl), TA, 0, s, act, apos, nl, alist);
+      GP_LAUNCH(g, k_bfs_sweep, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask, g->L, alist, apos + nl, bm,
+                levels, depth);
+    }
   }
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
@@ -102,33 +310,97 @@ __device__ __forceinline__ uint32_t cc_find(uint32_t *p, uint32_t x) {
   return cur;
 }
 
+__device__ __forceinline__ void cc_hook(uint32_t *p, uint32_t u, uint32_t v) {
+  uint32_t ru = cc_find(p, u), rv = cc_find(p, v);
+  bool repeat;
+  do {
+    repeat = false;
+    if (ru != rv) {
+      uint32_t ret;
+      if (ru < rv) {
+        if ((ret = atomicCAS(&p[rv], rv, ru)) != rv) { rv = ret; repeat = true; }
+      } else {
+        if ((ret = atomicCAS(&p[ru], ru, rv)) != ru) { ru = ret; repeat = true; }
+      }
+    }
+  } while (repeat);
+}
+
 __global__ void k_cc_init(uint32_t *p, uint32_t V) {
   for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
        v += (uint64_t)gridDim.x * blockDim.x)
     p[v] = (uint32_t)v;
 }
 
-__global__ void k_cc_hook(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val, uint64_t cap,
-                          uint32_t *p) {
-  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
-       s += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t k;
-    if (!edge_at(key, val, s, &k)) continue;
-    uint32_t u = (uint32_t)(k >> 32), v = (uint32_t)k;
-    if (u == v) continue;
-    uint32_t ru = cc_find(p, u), rv = cc_find(p, v);
-    bool repeat;
-    do {
-      repeat = false;
-      if (ru != rv) {
-        uint32_t ret;
-        if (ru < rv) {
-          if ((ret = atomicCAS(&p[rv], rv, ru)) != rv) { rv = ret; repeat = true; }
-        } else {
-          if ((ret = atomicCAS(&p[ru], ru, rv)) != ru) { ru = ret; repeat = true; }
-        }
-      }
-    } while (repeat);
+// Sample round: hook the first edge of every (source, leaf) run -- roughly the first one or
+// two edges of every row (Afforest-style neighbour sampling; any edge subset is a valid first
+// round), skipping pairs that already share a parent.
+__global__ void __launch_bounds__(TA) k_cc_sample(const uint64_t *__restrict__ key,
+                                                  const uint32_t *__restrict__ tmask, uint64_t cap, uint32_t L,
+                                                  uint32_t *p) {
+  const int lane = threadIdx.x & 31;
+  const uint64_t n4 = cap / 4, n4r = (n4 + 31) & ~31ull;
+  for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4r;
+       t += (uint64_t)gridDim.x * blockDim.x) {
+    Slot4 sl;
+    sl.k[0] = sl.k[1] = sl.k[2] = sl.k[3] = KEY_NONE;
+    sl.tb = 0;
+    if (t < n4) load4(key, tmask, L, t * 4, sl);
+    uint64_t prev = __shfl_up_sync(0xffffffffu, sl.k[3], 1);
+    if (lane == 0 && t < n4 && t > 0) prev = key[t * 4 - 1];
+    if (t >= n4) continue;
+#pragma unroll
+    for (int j = 0; j < 4; ++j) {
+      const uint64_t s = t * 4 + j;
+      const uint64_t pk = j ? sl.k[j - 1] : prev;
+      if (!edge4(sl, j)) continue;
+      const bool first = (s % L == 0) || pk == KEY_NONE || (pk >> 32) != (sl.k[j] >> 32);
+      if (!first) continue;
+      uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
+      if (u != v && __ldcg(p + u) != __ldcg(p + v)) cc_hook(p, u, v);
+    }
+  }
+}
+
+__global__ void k_cc_compress(uint32_t *p, uint32_t V) {
+  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
+       v += (uint64_t)gridDim.x * blockDim.x) {
+    volatile uint32_t *vp = p;
+    uint32_t x = vp[v], nx;
+    while ((nx = vp[x]) != x) x = nx;
+    vp[v] = x;
+  }
+}
+
+__device__ __forceinline__ void cc_group(const Slot4 &sl, uint32_t *p) {
+  uint32_t pu[4], pv[4];
+#pragma unroll
+  for (int j = 0; j < 4; ++j) {             // independent parent loads first
+    pu[j] = pv[j] = 0;
+    if (edge4(sl, j)) {
+      pu[j] = __ldcg(p + (uint32_t)(sl.k[j] >> 32));
+      pv[j] = __ldcg(p + (uint32_t)sl.k[j]);
+    }
+  }
+#pragma unroll
+  for (int j = 0; j < 4; ++j) {
+    if (!edge4(sl, j) || pu[j] == pv[j]) continue;   // same tree already (fast path)
+    uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
+    if (u != v) cc_hook(p, u, v);
+  }
+}
+
+__global__ void __launch_bounds__(TA) k_cc_hook(const uint64_t *__restrict__ key,
+                                                const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
+                                                uint32_t *p) {
+  const uint64_t n4 = cap / 4, stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4; t += 2 * stride) {
+    Slot4 a, b;
+    const bool hb = t + stride < n4;
+    load4(key, tmask, L, t * 4, a);
+    if (hb) load4(key, tmask, L, (t + stride) * 4, b);
+    cc_group(a, p);
+    if (hb) cc_group(b, p);
   }
 }
 
@@ -143,39 +415,19 @@ __global__ void k_cc_final(uint32_t *p, uint32_t *labels, uint32_t V) {
 }
 
 gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s) {
-  GP_CHECK(g, ensure(g->b_misc, ((uint64_t)g->V + 1) * 4, s));
-  uint32_t *p = (uint32_t *)g->b_misc.p;
+  GP_CHECK(g, ensure(g->b_an[0], ((uint64_t)g->V + 1) * 4, s));
+  uint32_t *p = (uint32_t *)g->b_an[0].p;
+  const uint32_t *tmask = tmask_of(g);
   GP_LAUNCH(g, k_cc_init, grid_for(g->V), TA, 0, s, p, g->V);
-  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap), TA, 0, s, g->key, g->val, g->cap, p);
+  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->cap, g->L, p);
+  GP_LAUNCH(g, k_cc_compress, grid_for(g->V), TA, 0, s, p, g->V);
+  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->L, g->cap, p);
   GP_LAUNCH(g, k_cc_final, grid_for(g->V), TA, 0, s, p, labels, g->V);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
 
 // ------------------------------------------------------------------ PageRank
-// out-degree of each row = live edges in it (warp-aggregated by source)
-__global__ void k_pr_outdeg(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val, uint64_t cap,
-                            uint32_t *deg) {
-  const int lane = threadIdx.x & 31;
-  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-  const uint64_t capr = (cap + 31) & ~31ull;
-  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < capr; s += stride) {
-    uint64_t k = 0;
-    bool e = s < cap && edge_at(key, val, s, &k);
-    uint32_t src = e ? (uint32_t)(k >> 32) : 0xFFFFFFFFu;
-    uint32_t peers = __match_any_sync(0xffffffffu, src);
-    if (e && (__ffs(peers) - 1) == lane) atomicAdd(&deg[src], (uint32_t)__popc(peers));
-  }
-}
-
-template <typename T>
-__global__ void k_pr_init(T *x, uint32_t V) {
-  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
-       v += (uint64_t)gridDim.x * blockDim.x)
-    x[v] = T(1) / T(V);
-}
-
-template <typename T>
 __device__ __forceinline__ double block_sum_d(double v, double *red) {
   for (int o = 16; o; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
   if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = v;
@@ -187,73 +439,133 @@ __device__ __forceinline__ double block_sum_d(double v, double *red) {
   return s;
 }
 
-// contrib[u] = x[u]/deg[u]; dangling mass D; y := 0
+// Accumulator of the push: exact fixed point for fp64 ranks, plain fp32 for the fp32 API.
 template <typename T>
-__global__ void k_pr_contrib(const T *__restrict__ x, const uint32_t *__restrict__ deg, T *__restrict__ contrib,
-                             T *__restrict__ y, uint32_t V, double *dsum) {
+struct PrAcc;
+template <>
+struct PrAcc<double> {
+  using A = unsigned long long;
+  static constexpr double SCALE = 4611686018427387904.0;   // 2^62
+  __device__ static A enc(double c) { return __double2ull_rn(c * SCALE); }
+  __device__ static double dec(A a) { return (double)a * (1.0 / SCALE); }
+};
+template <>
+struct PrAcc<float> {
+  using A = float;
+  __device__ static A enc(float c) { return c; }
+  __device__ static float dec(A a) { return a; }
+};
+
+// first iteration: x (given or 1/V), contrib = x/deg, dangling mass D, y = 0
+template <typename T>
+__global__ void k_pr_prep(T *__restrict__ x, const uint32_t *__restrict__ deg,
+                          typename PrAcc<T>::A *__restrict__ contrib, typename PrAcc<T>::A *__restrict__ y,
+                          uint32_t V, int init, double *dsum) {
   __shared__ double red[32];
   double dl = 0;
   for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
        v += (uint64_t)gridDim.x * blockDim.x) {
+    T xv = init ? T(1) / T(V) : x[v];
+    if (init) x[v] = xv;
     uint32_t dg = deg[v];
-    T xv = x[v];
-    contrib[v] = dg ? xv / T(dg) : T(0);
+    contrib[v] = PrAcc<T>::enc(dg ? xv / T(dg) : T(0));
     if (!dg) dl += (double)xv;
-    y[v] = T(0);
+    y[v] = 0;
   }
-  double s = block_sum_d<T>(dl, red);
+  double s = block_sum_d(dl, red);
   if (threadIdx.x == 0 && s != 0) atomicAdd(dsum, s);
 }
 
-template <typename T>
-__global__ void k_pr_push(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val, uint64_t cap,
-                          const T *__restrict__ contrib, T *y) {
-  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
-       s += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t k;
-    if (!edge_at(key, val, s, &k)) continue;
-    atomicAdd(&y[(uint32_t)k], contrib[k >> 32]);
+// y[v] += contrib[u] over the live edges u -> v (push SpMV): two groups of 4 slots per
+// thread, all loads (keys, masks, contributions) issued before the fire-and-forget REDs.
+template <typename A>
+__device__ __forceinline__ void pr_contribs(const Slot4 &sl, const A *__restrict__ contrib, A cv[4]) {
+  uint32_t cu = 0xFFFFFFFFu;
+  A c = 0;
+#pragma unroll
+  for (int j = 0; j < 4; ++j) {
+    cv[j] = 0;
+    if (!edge4(sl, j)) continue;
+    uint32_t u = (uint32_t)(sl.k[j] >> 32);
+    if (u != cu) { cu = u; c = __ldcs(contrib + u); }
+    cv[j] = c;
   }
 }
 
+template <typename A>
+__device__ __forceinline__ void pr_scatter(const Slot4 &sl, const A cv[4], A *y) {
+#pragma unroll
+  for (int j = 0; j < 4; ++j)
+    if (edge4(sl, j)) atomicAdd(&y[(uint32_t)sl.k[j]], cv[j]);
+}
+
+template <typename A>
+__global__ void __launch_bounds__(TA) k_pr_push(const uint64_t *__restrict__ key,
+                                                const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
+                                                const A *__restrict__ contrib, A *y) {
+  const uint64_t n4 = cap / 4, stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4; t += 2 * stride) {
+    Slot4 a, b;
+    const bool hb = t + stride < n4;
+    load4(key, tmask, L, t * 4, a);
+    if (hb) load4(key, tmask, L, (t + stride) * 4, b);
+    A ca[4], cb[4];
+    pr_contribs(a, contrib, ca);
+    if (hb) pr_contribs(b, contrib, cb);
+    pr_scatter(a, ca, y);
+    if (hb) pr_scatter(b, cb, y);
+  }
+}
+
+// x' = (1-d)/V + d (y + D/V); err += |x'-x|; next contrib / dangling; y := 0
 template <typename T>
-__global__ void k_pr_update(T *__restrict__ x, const T *__restrict__ y, uint32_t V, T d,
-                            const double *__restrict__ dsum, double *err) {
+__global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ y,
+                          const uint32_t *__restrict__ deg, typename PrAcc<T>::A *__restrict__ contrib,
+                          uint32_t V, T d, const double *__restrict__ dsum_in, double *dsum_out, double *err) {
   __shared__ double red[32];
-  const T base = (T(1) - d) / T(V) + d * T(*dsum / (double)V);
-  double e = 0;
+  const T base = (T(1) - d) / T(V) + d * T(*dsum_in / (double)V);
+  double e = 0, dl = 0;
   for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
        v += (uint64_t)gridDim.x * blockDim.x) {
-    T nx = base + d * y[v];
+    T nx = base + d * PrAcc<T>::dec(y[v]);
     e += fabs((double)nx - (double)x[v]);
     x[v] = nx;
+    y[v] = 0;
+    uint32_t dg = deg[v];
+    contrib[v] = PrAcc<T>::enc(dg ? nx / T(dg) : T(0));
+    if (!dg) dl += (double)nx;
   }
-  double s = block_sum_d<T>(e, red);
-  if (threadIdx.x == 0 && s != 0) atomicAdd(err, s);
+  double se = block_sum_d(e, red);
+  double sd = block_sum_d(dl, red);
+  if (threadIdx.x == 0) {
+    if (se != 0) atomicAdd(err, se);
+    if (sd != 0) atomicAdd(dsum_out, sd);
+  }
 }
 
 template <typename T>
 static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_iter, int *iters,
                               cudaStream_t s) {
+  using A = typename PrAcc<T>::A;
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(g->b_misc, (V + 1) * 4, s));
-  GP_CHECK(g, ensure(g->b_misc2, (V + 1) * sizeof(T), s));
-  GP_CHECK(g, ensure(g->b_misc3, (V + 1) * sizeof(T), s));
-  uint32_t *deg = (uint32_t *)g->b_misc.p;
-  T *contrib = (T *)g->b_misc2.p, *y = (T *)g->b_misc3.p;
-  double *dsum = (double *)&g->ctrl_d->sum;
-  double *err = (double *)&g->ctrl_d->sum2;
-  GP_CHECK(g, cudaMemsetAsync(deg, 0, V * 4, s));
-  GP_LAUNCH(g, k_pr_outdeg, grid_for(g->cap), TA, 0, s, g->key, g->val, g->cap, deg);
-  if (!warm) GP_LAUNCH(g, k_pr_init<T>, grid_for(V), TA, 0, s, x, (uint32_t)V);
-  int it = 0;
+  GP_CHECK(g, ensure(g->b_an[1], (V + 1) * sizeof(A), s));
+  GP_CHECK(g, ensure(g->b_an[2], (V + 1) * sizeof(A), s));
+  GP_CHECK(g, ensure(g->b_an[3], 4 * sizeof(double), s));
+  const uint32_t *deg = g->deg;
+  A *contrib = (A *)g->b_an[1].p, *y = (A *)g->b_an[2].p;
+  double *acc = (double *)g->b_an[3].p;   // [0],[1] dangling ping-pong, [2] error
+  GP_CHECK(g, cudaMemsetAsync(acc, 0, 4 * sizeof(double), s));
+  GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
+  int it = 0, cur = 0;
   while (it < max_iter) {
-    GP_CHECK(g, cudaMemsetAsync(&g->ctrl_d->sum, 0, 16, s));
-    GP_LAUNCH(g, k_pr_contrib<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, dsum);
-    GP_LAUNCH(g, k_pr_push<T>, grid_for(g->cap), TA, 0, s, g->key, g->val, g->cap, contrib, y);
-    GP_LAUNCH(g, k_pr_update<T>, grid_for(V), TA, 0, s, x, y, (uint32_t)V, d, dsum, err);
+    GP_LAUNCH(g, k_pr_push<A>, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, contrib, y);
+    GP_CHECK(g, cudaMemsetAsync(acc + 2, 0, sizeof(double), s));
+    GP_CHECK(g, cudaMemsetAsync(acc + (cur ^ 1), 0, sizeof(double), s));
+    GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
+              acc + (cur ^ 1), acc + 2);
+    cur ^= 1;
     ++it;
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, &g->ctrl_d->sum2, 8, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, acc + 2, 8, cudaMemcpyDeviceToHost, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
     double e;
     memcpy(&e, &g->ctrl_h->sum2, 8);
@@ -275,35 +587,63 @@ gpma_status pagerank_f32(gpma *g, float *x, int warm, float d, float tol, int ma
 }
 
 // ------------------------------------------------------------------ export CSR
-__global__ void k_exp_leafcount(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val,
-                                uint32_t L, uint64_t nleaves, uint64_t *lc) {
-  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
-       l += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t c = 0, k;
-    for (uint32_t p = 0; p < L; ++p) c += edge_at(key, val, l * L + p, &k);
-    lc[l] = c;
+// guards per leaf from the row offsets (R8: row_offset[u+1] = slot of guard u)
+__global__ void k_exp_guards(const uint64_t *__restrict__ row_offset, const uint64_t *__restrict__ key,
+                             uint32_t V, uint32_t L, uint32_t *__restrict__ gl) {
+  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < V;
+       u += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t s = row_offset[u + 1];
+    if (key[s] == ((u << 32) | COL_GUARD)) atomicAdd(&gl[s / L], 1u);
   }
 }
 
-__global__ void k_exp_write(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val, uint32_t L,
-                            uint64_t cap, const uint64_t *__restrict__ lbase, uint64_t *__restrict__ row_ptr,
-                            uint32_t *__restrict__ col, uint32_t *__restrict__ cval) {
+// edges per leaf = live entries (cnt) - guards
+__global__ void k_exp_counts(const uint32_t *__restrict__ cnt, const uint32_t *__restrict__ gl, uint64_t nl,
+                             uint64_t *__restrict__ lc) {
+  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nl;
+       l += (uint64_t)gridDim.x * blockDim.x)
+    lc[l] = cnt[l] - gl[l];
+}
+
+// Compaction sweep, 4 slots per thread: rank = leaf base + edges before this slot in the
+// leaf (exclusive scan over the L/4 lanes that share the leaf + the thread's own slots).
+__global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ key,
+                                                  const uint32_t *__restrict__ val,
+                                                  const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
+                                                  const uint64_t *__restrict__ lbase,
+                                                  uint64_t *__restrict__ row_ptr, uint32_t *__restrict__ col,
+                                                  uint32_t *__restrict__ cval) {
   const int lane = threadIdx.x & 31;
-  const uint32_t lt = (1u << lane) - 1u;
-  const uint32_t leafmask = (L == 32 ? 0xffffffffu : ((1u << L) - 1u) << (lane & ~(L - 1)));
-  const uint64_t capr = (cap + 31) & ~31ull;
-  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < capr;
-       s += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t k = KEY_NONE;
-    bool e = s < cap && edge_at(key, val, s, &k);
-    uint32_t bal = __ballot_sync(0xffffffffu, e);
-    if (s >= cap) continue;
-    uint64_t r = lbase[s / L] + __popc(bal & leafmask & lt);
-    if (e) {
-      col[r] = (uint32_t)k;
-      cval[r] = val[s];
-    } else if (is_guard_key(k)) {
-      row_ptr[(k >> 32) + 1] = r;
+  const uint32_t lpl = L / 4;                    // lanes per leaf (1..8)
+  const uint64_t n4 = cap / 4, n4r = (n4 + 31) & ~31ull;
+  for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4r;
+       t += (uint64_t)gridDim.x * blockDim.x) {
+    Slot4 sl;
+    uint32_t e = 0;
+    if (t < n4) {
+      load4(key, tmask, L, t * 4, sl);
+#pragma unroll
+      for (int j = 0; j < 4; ++j) e |= (edge4(sl, j) ? 1u : 0u) << j;
+    }
+    uint32_t c = __popc(e), incl = c;
+    for (uint32_t o = 1; o < lpl; o <<= 1) {
+      uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+      if ((lane % lpl) >= o) incl += y;
+    }
+    if (t >= n4) continue;
+    uint64_t r = lbase[(t * 4) / L] + incl - c;
+    uint4 vv = make_uint4(0, 0, 0, 0);
+    if (e) vv = __ldcs(reinterpret_cast<const uint4 *>(val + t * 4));
+    const uint32_t vs[4] = {vv.x, vv.y, vv.z, vv.w};
+#pragma unroll
+    for (int j = 0; j < 4; ++j) {
+      if ((e >> j) & 1u) {
+        col[r] = (uint32_t)sl.k[j];
+        cval[r] = vs[j];
+        ++r;
+      } else if (is_guard_key(sl.k[j])) {
+        row_ptr[(sl.k[j] >> 32) + 1] = r;
+      }
     }
   }
 }
@@ -312,8 +652,12 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
                        uint64_t *nnz_out, cudaStream_t s) {
   const uint64_t nl = g->cap / g->L;
   GP_CHECK(g, ensure(g->b_lpre, (nl + 1) * 8, s));
+  GP_CHECK(g, ensure(g->b_an[0], (nl + 1) * 4, s));
   uint64_t *lc = (uint64_t *)g->b_lpre.p;
-  GP_LAUNCH(g, k_exp_leafcount, grid_for(nl), TA, 0, s, g->key, g->val, g->L, nl, lc);
+  uint32_t *gl = (uint32_t *)g->b_an[0].p;
+  GP_CHECK(g, cudaMemsetAsync(gl, 0, nl * 4, s));
+  GP_LAUNCH(g, k_exp_guards, grid_for(g->V), TA, 0, s, g->row_offset, g->key, g->V, g->L, gl);
+  GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gl, nl, lc);
   scan_u64(g, lc, lc, nl, s);
   GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, lc + nl, 8, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
@@ -325,8 +669,8 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
     return GPMA_ERR_INVALID_ARG;
   }
   GP_CHECK(g, cudaMemsetAsync(row_ptr, 0, 8, s));
-  GP_LAUNCH(g, k_exp_write, grid_for(g->cap), TA, 0, s, g->key, g->val, g->L, g->cap, lc, row_ptr, col,
-            val);
+  GP_LAUNCH(g, k_exp_write, grid_for(g->cap / 4), TA, 0, s, g->key, g->val, tmask_of(g), g->L, g->cap, lc,
+            row_ptr, col, val);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }

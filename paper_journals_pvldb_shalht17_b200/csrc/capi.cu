@@ -118,13 +118,15 @@ void free_handle(gpma *g) {
                     &g->b_hf, &g->b_widx, &g->b_wfirst, &g->b_acc, &g->b_aidx, &g->b_alist, &g->b_nw,
                     &g->b_woff, &g->b_keep2, &g->b_kpos, &g->b_lpre, &g->b_wk, &g->b_wv, &g->b_dirty,
                     &g->b_scan, &g->b_hist, &g->b_stage[0], &g->b_stage[1], &g->b_stage[2],
-                    &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3};
+                    &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3,
+                    &g->b_an[0], &g->b_an[1], &g->b_an[2], &g->b_an[3]};
   for (DevBuf *b : bufs) gp::release(*b, s);
   if (g->key) cudaFreeAsync(g->key, s);
   if (g->val) cudaFreeAsync(g->val, s);
   if (g->cnt) cudaFreeAsync(g->cnt, s);
   if (g->head) cudaFreeAsync(g->head, s);
   if (g->row_offset) cudaFreeAsync(g->row_offset, s);
+  if (g->deg) cudaFreeAsync(g->deg, s);
   cudaStreamSynchronize(s);
   for (cudaEvent_t e : g->ev_pool) cudaEventDestroy(e);
   if (g->ctrl_d) cudaFree(g->ctrl_d);
@@ -203,8 +205,9 @@ gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t l
     gp::level_bounds(g->L, g->h, g->rho0, g->rhoh, g->tau0, g->tauh, g->tmin, g->tmax);
     uint64_t nl = capacity / leaf_slots;
     if (cudaMallocAsync((void **)&g->key, capacity * 8, s) || cudaMallocAsync((void **)&g->val, capacity * 4, s) ||
-        cudaMallocAsync((void **)&g->cnt, nl * 4, s) || cudaMallocAsync((void **)&g->head, nl * 8, s) ||
-        cudaMallocAsync((void **)&g->row_offset, ((uint64_t)num_vertices + 1) * 8, s)) {
+        cudaMallocAsync((void **)&g->cnt, nl * 8, s) || cudaMallocAsync((void **)&g->head, nl * 8, s) ||
+        cudaMallocAsync((void **)&g->row_offset, ((uint64_t)num_vertices + 1) * 8, s) ||
+        cudaMallocAsync((void **)&g->deg, (uint64_t)num_vertices * 4, s)) {
       cudaGetLastError();
       st = GPMA_ERR_OOM;
     }

@@ -64,7 +64,9 @@ struct gpma {
   // store (HBM-resident)
   uint64_t *key = nullptr;        // [cap]
   uint32_t *val = nullptr;        // [cap]
-  uint32_t *cnt = nullptr;        // [cap/L] live entries (incl. guards) per leaf
+  uint32_t *cnt = nullptr;        // [2*cap/L]: live entries (incl. guards) per leaf, then the
+                                  // per-leaf tombstone bit mask (bit p = slot p is a tombstone)
+  uint32_t *deg = nullptr;        // [V] live out-degree per vertex, maintained by every batch
   uint64_t *head = nullptr;       // [cap/L] locate index (R9)
   uint64_t *row_offset = nullptr; // [V+1] (R8)
 
@@ -73,6 +75,7 @@ struct gpma {
   gp::DevBuf b_pk[2], b_pv[2], b_pt[2];                      // pending (ping-pong)
   gp::DevBuf b_hf, b_widx, b_wfirst, b_acc, b_aidx, b_alist, b_nw, b_woff, b_keep2, b_kpos;
   gp::DevBuf b_lpre, b_wk, b_wv, b_dirty, b_scan, b_hist, b_stage[4], b_misc, b_misc2, b_misc3;
+  gp::DevBuf b_an[4];                                           // analytics scratch
   gp::Ctrl *ctrl_d = nullptr;
   gp::Ctrl *ctrl_h = nullptr;     // pinned mirror
 
@@ -145,6 +148,8 @@ gpma_status build_from_sorted(gpma *g, const uint64_t *sk, const uint32_t *sv, u
 gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaStream_t s);
 gpma_status recompute_heads(gpma *g, cudaStream_t s);
 gpma_status count_slots(gpma *g, uint64_t *live_edges, uint64_t *tombs, cudaStream_t s);
+gpma_status recompute_degrees(gpma *g, cudaStream_t s);   // analytics.cu
+inline uint32_t *tmask_of(gpma *g) { return g->cnt + g->cap / g->L; }
 
 // analytics (analytics.cu)
 gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s);

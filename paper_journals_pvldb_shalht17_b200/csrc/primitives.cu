@@ -114,7 +114,6 @@ int key_shifts(uint32_t V, int *shifts) {
 constexpr int SC_THREADS = 256;
 constexpr int SC_ITEMS = 16;
 constexpr int SC_TILE = SC_THREADS * SC_ITEMS;   // 4096
-constexpr uint64_t SC_SINGLE_MAX = 1 << 16;
 
 template <typename T>
 __device__ __forceinline__ T warp_sum(T x) {
@@ -133,112 +132,93 @@ __device__ __forceinline__ T warp_incl_scan(T x, int lane) {
   return x;
 }
 
+// Single-pass scan with decoupled look-back: each CTA takes the next tile id from a
+// counter, publishes its aggregate, then walks back over its predecessors' published
+// (aggregate | inclusive) values until it meets an inclusive prefix.  Status word:
+// flag in bits 62-63 (0 = not ready, 1 = aggregate, 2 = inclusive), value below.
 template <typename T>
-__global__ void k_scan_single(const T *__restrict__ in, T *__restrict__ out, uint64_t n) {
-  __shared__ T wsum[32];
-  __shared__ T carry_s;
-  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  if (threadIdx.x == 0) carry_s = 0;
-  __syncthreads();
-  for (uint64_t base = 0; base < n; base += blockDim.x) {
-    uint64_t i = base + threadIdx.x;
-    T x = i < n ? in[i] : T(0);
-    T inc = warp_incl_scan(x, lane);
-    if (lane == 31) wsum[w] = inc;
-    __syncthreads();
-    if (w == 0) {
-      T s = lane < (int)(blockDim.x >> 5) ? wsum[lane] : T(0);
-      T si = warp_incl_scan(s, lane);
-      wsum[lane] = si - s;
-    }
-    __syncthreads();
-    T c = carry_s;
-    if (i < n) out[i] = c + wsum[w] + inc - x;
-    __syncthreads();
-    if (threadIdx.x == blockDim.x - 1) carry_s = c + wsum[w] + inc;
-    __syncthreads();
-  }
-  if (threadIdx.x == 0) out[n] = carry_s;
-}
-
-template <typename T>
-__global__ void k_scan_reduce(const T *__restrict__ in, T *__restrict__ partial, uint64_t n) {
+__global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *out, uint64_t n,
+                                                               unsigned long long *status) {
+  __shared__ uint32_t s_tile;
   __shared__ T ws[SC_THREADS / 32];
-  const uint64_t base = (uint64_t)blockIdx.x * SC_TILE;
-  T s = 0;
-#pragma unroll
-  for (int j = 0; j < SC_ITEMS; ++j) {
-    uint64_t i = base + (uint64_t)j * SC_THREADS + threadIdx.x;
-    if (i < n) s += in[i];
-  }
-  s = warp_sum(s);
-  if ((threadIdx.x & 31) == 0) ws[threadIdx.x >> 5] = s;
-  __syncthreads();
-  if (threadIdx.x < 32) {
-    T t = threadIdx.x < SC_THREADS / 32 ? ws[threadIdx.x] : T(0);
-    t = warp_sum(t);
-    if (threadIdx.x == 0) partial[blockIdx.x] = t;
-  }
-}
-
-template <typename T>
-__global__ void k_scan_down(const T *in, T *out, const T *__restrict__ partial, uint64_t n,
-                            uint64_t nb) {
-  __shared__ T ws[SC_THREADS / 32];
+  __shared__ T s_prefix;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  const uint64_t base = (uint64_t)blockIdx.x * SC_TILE + (uint64_t)w * (32 * SC_ITEMS);
-  T s = 0;
+  if (threadIdx.x == 0) s_tile = (uint32_t)atomicAdd(status, 1ull);  // status[0] = tile counter
+  __syncthreads();
+  const uint32_t tile = s_tile;
+  volatile unsigned long long *st = status + 1;
+  const uint64_t base = (uint64_t)tile * SC_TILE + (uint64_t)w * (32 * SC_ITEMS);
+  T x[SC_ITEMS];
+  T part = 0;
 #pragma unroll
   for (int j = 0; j < SC_ITEMS; ++j) {
     uint64_t i = base + j * 32 + lane;
-    if (i < n) s += in[i];
+    x[j] = i < n ? in[i] : T(0);
+    part += x[j];
   }
-  s = warp_sum(s);
-  if (lane == 0) ws[w] = s;
+  T wtot = warp_sum(part);
+  if (lane == 0) ws[w] = wtot;
   __syncthreads();
-  T carry = partial[blockIdx.x];
+  if (w == 0) {
+    T agg = 0;
+    for (int k = 0; k < SC_THREADS / 32; ++k) agg += ws[k];
+    const unsigned long long VMASK = (1ull << 62) - 1;
+    T prefix = 0;
+    if (lane == 0) {
+      __threadfence();
+      st[tile] = ((tile == 0 ? 2ull : 1ull) << 62) | ((unsigned long long)agg & VMASK);
+    }
+    // warp-parallel look-back over windows of 32 predecessors
+    int64_t t = (int64_t)tile - 1;
+    while (t >= 0) {
+      int64_t mine = t - lane;
+      unsigned long long v = 2ull << 62;        // lanes past tile 0 act as an inclusive zero
+      if (mine >= 0) {
+        do { v = st[mine]; } while ((v >> 62) == 0);
+      }
+      uint32_t inc = __ballot_sync(0xffffffffu, (v >> 62) == 2);
+      int stop = inc ? __ffs(inc) - 1 : 31;     // nearest predecessor with an inclusive prefix
+      T contrib = (lane <= stop) ? (T)(v & VMASK) : T(0);
+      prefix += warp_sum(contrib);
+      if (inc) break;
+      t -= 32;
+    }
+    if (lane == 0) {
+      if (tile) {
+        __threadfence();
+        st[tile] = (2ull << 62) | ((unsigned long long)(prefix + agg) & VMASK);
+      }
+      s_prefix = prefix;
+      if ((uint64_t)(tile + 1) * SC_TILE >= n) out[n] = prefix + agg;   // last tile: total
+    }
+  }
+  __syncthreads();
+  T carry = s_prefix;
   for (int k = 0; k < w; ++k) carry += ws[k];
 #pragma unroll
   for (int j = 0; j < SC_ITEMS; ++j) {
     uint64_t i = base + j * 32 + lane;
-    T x = i < n ? in[i] : T(0);
-    T inc = warp_incl_scan(x, lane);
-    if (i < n) out[i] = carry + inc - x;
+    T inc = warp_incl_scan(x[j], lane);
+    if (i < n) out[i] = carry + inc - x[j];
     carry += __shfl_sync(0xffffffffu, inc, 31);
   }
-  if (blockIdx.x == 0 && threadIdx.x == 0) out[n] = partial[nb];
 }
 
 template <typename T>
-static void scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s, T *tmp) {
-  if (n <= SC_SINGLE_MAX) {
-    GP_LAUNCH(g, k_scan_single<T>, 1, 1024, 0, s, in, out, n);
-    return;
-  }
-  uint64_t nb = (n + SC_TILE - 1) / SC_TILE;
-  T *partial = tmp;
-  GP_LAUNCH(g, k_scan_reduce<T>, (unsigned)nb, SC_THREADS, 0, s, in, partial, n);
-  scan_impl<T>(g, partial, partial, nb, s, tmp + nb + 1);
-  GP_LAUNCH(g, k_scan_down<T>, (unsigned)nb, SC_THREADS, 0, s, in, out, partial, n, nb);
-}
-
-static size_t scan_tmp_elems(uint64_t n) {
-  size_t t = 0;
-  while (n > SC_SINGLE_MAX) {
-    n = (n + SC_TILE - 1) / SC_TILE;
-    t += n + 1;
-  }
-  return t + 1;
+static void scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) {
+  const uint64_t nt = (n + SC_TILE - 1) / SC_TILE > 0 ? (n + SC_TILE - 1) / SC_TILE : 1;
+  ensure(g->b_scan, (nt + 1) * sizeof(unsigned long long), s);
+  unsigned long long *status = (unsigned long long *)g->b_scan.p;
+  cudaMemsetAsync(status, 0, (nt + 1) * sizeof(unsigned long long), s);
+  GP_LAUNCH(g, k_scan_lookback<T>, (unsigned)nt, SC_THREADS, 0, s, in, out, n, status);
 }
 
 void scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s) {
-  ensure(g->b_scan, scan_tmp_elems(n) * sizeof(uint64_t), s);
-  scan_impl<uint32_t>(g, in, out, n, s, (uint32_t *)g->b_scan.p);
+  scan_impl<uint32_t>(g, in, out, n, s);
 }
 
 void scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s) {
-  ensure(g->b_scan, scan_tmp_elems(n) * sizeof(uint64_t), s);
-  scan_impl<uint64_t>(g, in, out, n, s, (uint64_t *)g->b_scan.p);
+  scan_impl<uint64_t>(g, in, out, n, s);
 }
 
 // ------------------------------------------------------------------ radix sort
@@ -247,7 +227,7 @@ void scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream
 // exclusive scan over the digit-major (digit, tile) table -> stable scatter, where
 // the rank inside a tile comes from __match_any_sync peer groups per warp round.
 constexpr int RS_THREADS = 256;
-constexpr int RS_ITEMS = 16;
+constexpr int RS_ITEMS = 8;
 constexpr int RS_WARPS = RS_THREADS / 32;
 constexpr int RS_TILE = RS_THREADS * RS_ITEMS;
 

@@ -57,7 +57,8 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
                           uint64_t n, const uint64_t *__restrict__ key, uint32_t *__restrict__ val,
                           uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
                           uint32_t nleaves, uint32_t L, int op, int mode,
-                          uint32_t *__restrict__ keep, uint32_t *__restrict__ tgt, Ctrl *c) {
+                          uint32_t *__restrict__ keep, uint32_t *__restrict__ tgt, Ctrl *c,
+                          uint32_t *__restrict__ tmask, uint32_t *__restrict__ deg) {
   uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
   uint32_t uniq = 0;
   if (i < n) {
@@ -72,21 +73,33 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
         if (x == k) { hit = base + p; break; }
         if (x == KEY_NONE || x > k) break;
       }
+      const uint32_t src = (uint32_t)(k >> 32);
+      const uint32_t bit = hit != KEY_NONE ? 1u << (uint32_t)(hit - base) : 0u;
       if (op == GPMA_INSERT) {
         if (hit != KEY_NONE) {                      // overwrite (R11) or revive (R12)
           uint32_t old = val[hit];
           val[hit] = sv[i];
-          if (old == VAL_TOMB) atomicAdd(&cnt[t], 1u);
+          if (old == VAL_TOMB) {
+            atomicAdd(&cnt[t], 1u);
+            atomicAnd(&tmask[t], ~bit);
+            atomicAdd(&deg[src], 1u);
+          }
         } else {
-          kp = 1;
+          kp = 1;                                   // new key: inserted by the level loop
+          atomicAdd(&deg[src], 1u);
         }
       } else if (mode == GPMA_DELETE_LAZY) {        // mark, no maintenance
         if (hit != KEY_NONE && val[hit] != VAL_TOMB) {
           val[hit] = VAL_TOMB;
           atomicSub(&cnt[t], 1u);
+          atomicOr(&tmask[t], bit);
+          atomicSub(&deg[src], 1u);
         }
       } else {                                      // strict delete: live keys only
-        if (hit != KEY_NONE && val[hit] != VAL_TOMB) kp = 1;
+        if (hit != KEY_NONE && val[hit] != VAL_TOMB) {
+          kp = 1;
+          atomicSub(&deg[src], 1u);
+        }
       }
     }
     keep[i] = kp;
@@ -304,8 +317,9 @@ __global__ void k_lvl_place(Lvl a, const uint64_t *__restrict__ key, const uint3
 // entries receives entries [floor(l N / Lc), floor((l+1) N / Lc)), left-packed.
 // Guards moved here update the row offsets (R8).
 __global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
-                                   uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset,
-                                   uint64_t bound, uint2 *__restrict__ dirty, uint64_t dirty_base) {
+                                   uint32_t *__restrict__ cnt, uint32_t *__restrict__ tmask,
+                                   uint64_t *__restrict__ row_offset, uint64_t bound,
+                                   uint2 *__restrict__ dirty, uint64_t dirty_base) {
   const uint32_t nacc = a.aidx[a.p];
   const uint64_t Lc = 1ull << a.lvl;
   const uint64_t wslots = (uint64_t)a.L << a.lvl;
@@ -330,7 +344,10 @@ __global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *
       key[s] = KEY_NONE;
       val[s] = 0;
     }
-    if (p == 0) cnt[leaf0 + l] = (uint32_t)(hi - lo);
+    if (p == 0) {
+      cnt[leaf0 + l] = (uint32_t)(hi - lo);
+      tmask[leaf0 + l] = 0u;                          // tombstones are dropped by a rewrite
+    }
     if (off == 0) dirty[dirty_base + ai] = make_uint2((uint32_t)leaf0, (uint32_t)Lc);
   }
 }
@@ -354,6 +371,7 @@ __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *_
                               uint64_t N, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
                               uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset,
                               uint32_t L, uint64_t nleaves) {
+  uint32_t *tmask = cnt + nleaves;
   const uint64_t cap = nleaves * L;
   for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
        s += (uint64_t)gridDim.x * blockDim.x) {
@@ -368,7 +386,10 @@ __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *_
       key[s] = KEY_NONE;
       val[s] = 0;
     }
-    if (p == 0) cnt[l] = (uint32_t)(hi - lo);
+    if (p == 0) {
+      cnt[l] = (uint32_t)(hi - lo);
+      tmask[l] = 0u;
+    }
   }
 }
 
@@ -492,15 +513,17 @@ __global__ void k_raw_counts(const uint64_t *__restrict__ key, const uint32_t *_
                              uint64_t nleaves, uint32_t V) {
   for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
        l += (uint64_t)gridDim.x * blockDim.x) {
-    uint32_t c = 0;
+    uint32_t c = 0, m = 0;
     for (uint32_t p = 0; p < L; ++p) {
       uint64_t s = l * L + p;
       uint64_t k = key[s];
       if (k == KEY_NONE) continue;
       if (val[s] != VAL_TOMB) ++c;
+      else m |= 1u << p;
       if (is_guard_key(k) && (k >> 32) < V) row_offset[(k >> 32) + 1] = s;
     }
     cnt[l] = c;
+    cnt[nleaves + l] = m;
   }
 }
 
@@ -545,7 +568,7 @@ static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v
   *k = nullptr; *v = nullptr; *c = nullptr; *hd = nullptr;
   cudaError_t e1 = cudaMallocAsync((void **)k, cap * 8, s);
   cudaError_t e2 = cudaMallocAsync((void **)v, cap * 4, s);
-  cudaError_t e3 = cudaMallocAsync((void **)c, nl * 4, s);
+  cudaError_t e3 = cudaMallocAsync((void **)c, nl * 8, s);   // live counts + tombstone masks
   cudaError_t e4 = cudaMallocAsync((void **)hd, nl * 8, s);
   if (e1 || e2 || e3 || e4) {
     cudaGetLastError();
@@ -566,7 +589,9 @@ gpma_status build_from_sorted(gpma *g, const uint64_t *wk, const uint32_t *wv, u
   GP_LAUNCH(g, k_layout_even, grid_for(g->cap), TB, 0, s, wk, wv, N, g->key, g->val, g->cnt,
             g->row_offset, g->L, nl);
   GP_CHECK(g, cudaGetLastError());
-  return recompute_heads(g, s);
+  gpma_status st = recompute_heads(g, s);
+  if (st) return st;
+  return recompute_degrees(g, s);
 }
 
 gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaStream_t s) {
@@ -576,7 +601,9 @@ gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaSt
   GP_LAUNCH(g, k_raw_counts, grid_for(nl), TB, 0, s, g->key, g->val, g->cnt, g->row_offset, g->L, nl,
             g->V);
   GP_CHECK(g, cudaGetLastError());
-  return recompute_heads(g, s);
+  gpma_status st = recompute_heads(g, s);
+  if (st) return st;
+  return recompute_degrees(g, s);
 }
 
 // Sort a device batch (keys, vals) of n pairs and drop all but the last copy of each
@@ -669,6 +696,7 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
   if ((st = alloc_store(g, cap, &g->key, &g->val, &g->cnt, &g->head, s))) return st;
   GP_CHECK(g, cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->V + 1) * 8, s));
   GP_CHECK(g, cudaMemsetAsync(g->row_offset, 0, ((uint64_t)g->V + 1) * 8, s));
+  GP_CHECK(g, cudaMallocAsync((void **)&g->deg, (uint64_t)g->V * 4, s));
   if (E > g->tmax[g->h] && !cap_override) {
     g->err = "initial graph exceeds the root bound";
     return GPMA_ERR_INVALID_ARG;
@@ -734,7 +762,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   GP_LAUNCH(g, k_lvl_gather, grid_for(bslots_r), TB, 0, s, a, g->key, g->val, bslots_r);
   if (a.op == GPMA_INSERT) GP_LAUNCH(g, k_lvl_place, gp, TB, 0, s, a, g->key, g->val);
   if (!resize_target) {
-    GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots), TB, 0, s, a, g->key, g->val, g->cnt,
+    GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots), TB, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
               g->row_offset, bslots, (uint2 *)g->b_dirty.p, *dirty_base);
   } else {
     // the single root window, laid out over the whole new array
@@ -912,7 +940,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   if ((st = zero_ctrl(g, s))) return st;
   const uint64_t nl = g->cap / g->L;
   GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt,
-            g->head, (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d);
+            g->head, (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg);
   scan_u32(g, keep, pos, n, s);
   GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, pos + n, 4, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->nunique, &g->ctrl_d->nunique, 8, cudaMemcpyDeviceToHost, s));
