@@ -280,6 +280,11 @@ def run_gpma(args, rank, world, lrank):
     hbm, peak_kind = peaks()
     nnz = st["live_edges"]
     ab = algo_bytes(dom, cap, V, st["leaf_slots"], nnz)
+    traffic = None
+    tpath = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    if os.path.exists(tpath):
+        with open(tpath) as f:
+            traffic = json.load(f).get("dram_bytes_per_launch", {}).get(dom)
     n_l, tot_ms = prof_dom
     avg_ms = tot_ms / n_l if n_l else float("nan")
     achieved = ab / (avg_ms / 1e3) / 1e9 if n_l else None
@@ -307,7 +312,8 @@ def run_gpma(args, rank, world, lrank):
                         "ms_per_slide": phase_ms[0] + phase_ms[1]},
         "pr_iters": iters_timed,
         "roofline": {"bound": "hbm", "kernel": dom, "achieved": achieved, "peak": hbm, "unit": "GB/s",
-                     "frac": (achieved / hbm) if achieved else None, "traffic": None,
+                     "frac": (achieved / hbm) if achieved else None, "traffic": traffic,
+                     "traffic_source": "profiles/ncu_traffic.json (ncu --set full, dram read+write per launch)",
                      "algorithmic_bytes_per_launch": ab, "avg_launch_ms": avg_ms, "launches": n_l,
                      "peak_kind": peak_kind},
         "e2e": e2e,
