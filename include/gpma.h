@@ -68,6 +68,10 @@ typedef struct {
   uint16_t init_density_bp;   /* R15: 6000                                            */
   uint16_t reserved0;
   uint32_t delete_mode;       /* gpma_delete_mode                                     */
+  uint32_t row_begin, row_end;/* shard (R24): the store holds the rows
+                                 (sources) [row_begin, row_end) only -- guards, row
+                                 offsets and out-degrees for those rows; destinations
+                                 range over [0, num_vertices).  0,0 = all rows.       */
 } gpma_config;
 
 typedef struct {
@@ -156,6 +160,40 @@ gpma_status gpma_debug_set_trace(gpma_t *g, int enable);
 /* Records (level, seg_start_slot, offset, flag) x4 u64; flag 2 closes a level and
  * carries the final offset.  Returns the record count in *count; copies at most max. */
 gpma_status gpma_debug_trace(gpma_t *g, uint64_t *out4, uint64_t max, uint64_t *count);
+
+/* ---------------------------------------------------------------- sharded stores
+ * Multi-GPU ("evenly partition graphs according to the vertex index and
+ * synchronize all devices after each iteration"; R24): one store per rank holds
+ * the rows [row_begin, row_end) of owner(u) = u / ceil(V / P) (gpma_config.row_begin/end).
+ * The primitives below are the per-rank steps between the collectives of a distributed
+ * update / BFS / CC / PageRank (the caller, e.g. paper_journals_pvldb_shalht17_b200.dist,
+ * runs the collectives).  All their array arguments are DEVICE pointers. */
+
+/* Stable partition of a batch slice by owner rank: out_keys/out_vals (n each) hold the
+ * owner-0 keys, then owner-1, ...; counts[nranks] (HOST) the piece sizes.  vals may be NULL
+ * (zeros are routed).  Works on any handle (only V is used). */
+gpma_status gpma_route(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, uint32_t nranks,
+                       uint64_t *out_keys, uint32_t *out_vals, uint64_t *counts, gpma_stream_t stream);
+
+/* levels[V] := -1, levels[root] := 0. */
+gpma_status gpma_bfs_init(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t stream);
+/* One BFS level (Alg. 3 over the owned rows): frontier = {v : levels[v] == depth-1};
+ * unreached out-neighbours of the owned frontier rows get `depth`.  *frontier_size (HOST) =
+ * |frontier| (0: done).  Combine shards with an element-wise MAX of levels between levels. */
+gpma_status gpma_bfs_level(gpma_t *g, int32_t *levels, int32_t depth, uint32_t *frontier_size,
+                           gpma_stream_t stream);
+/* One CC round over the owned edges on top of labels[V] (a forest with labels[x] <= x;
+ * init != 0 starts from the identity): hook + compress.  *changed (HOST) = labels moved.
+ * Combine shards with an element-wise MIN; the fixpoint (no shard changes) is the min-id
+ * labelling of the weak components (R19). */
+gpma_status gpma_cc_round(gpma_t *g, uint32_t *labels, int init, uint64_t *changed, gpma_stream_t stream);
+/* PageRank push over the owned rows: x[V] (replicated; init != 0 sets 1/V first) ->
+ * y[0..V) += sum over owned edges u->v of x[u]/outdeg(u), y[V] += dangling mass of the owned
+ * rows; y is 64-bit fixed point with 2^-62 units.  Combine shards with a SUM of y. */
+gpma_status gpma_pr_push(gpma_t *g, double *x, int init, uint64_t *y, gpma_stream_t stream);
+/* x'[v] = (1-d)/V + d*(y[v] + y[V]/V) for every v; *err (HOST) = ||x'-x||_1; y := 0. */
+gpma_status gpma_pr_update(gpma_t *g, double *x, uint64_t *y, double damping, double *err,
+                           gpma_stream_t stream);
 
 /* Kernel profiler (bench evidence, CUDA events on the call's stream around each launch):
  * filter NULL/"" = off, "*" = every kernel, else one kernel name (e.g. "k_pr_push").

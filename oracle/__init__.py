@@ -48,6 +48,7 @@ def lib():
         sig = {
             "orc_create": (P, [u32, P, P, u64, u32, u64, i32, P]),
             "orc_create_raw": (P, [u32, u64, u32, P, P, i32, P]),
+            "orc_create_shard": (P, [u32, u32, u32, P, P, u64, u32, u64, i32, P]),
             "orc_destroy": (None, [P]),
             "orc_update": (i32, [P, P, P, u64, i32]),
             "orc_capacity": (u64, [P]),
@@ -116,7 +117,7 @@ class Oracle:
     """One sequential GPMA+ store."""
 
     def __init__(self, V: int, keys=(), vals=(), *, leaf_slots: int = 0, capacity: int = 0,
-                 delete_mode: int = LAZY, _raw=None):
+                 delete_mode: int = LAZY, rows=None, _raw=None):
         st = C.c_int(0)
         if _raw is not None:
             cap, L, rk, rv = _raw
@@ -124,11 +125,13 @@ class Oracle:
             self._h = lib().orc_create_raw(V, cap, L, _p(rk), _p(rv), delete_mode, C.byref(st))
         else:
             k, v = _u64(keys), _u32(vals)
-            self._h = lib().orc_create(V, _p(k), _p(v), k.size, leaf_slots, capacity, delete_mode,
-                                       C.byref(st))
+            rb, re = rows if rows is not None else (0, 0)
+            self._h = lib().orc_create_shard(V, rb, re, _p(k), _p(v), k.size, leaf_slots, capacity,
+                                             delete_mode, C.byref(st))
         if st.value != OK:
             raise OracleError(st.value)
         self.V = V
+        self.rb, self.nr = (rows[0], rows[1] - rows[0]) if rows is not None and rows[1] > rows[0] else (0, V)
 
     @classmethod
     def raw(cls, V, cap, L, keys, vals=None, delete_mode=LAZY):
@@ -163,7 +166,7 @@ class Oracle:
         out = np.zeros(16, np.uint64)
         lib().orc_stats(self._h, _p(out))
         names = ["cap", "L", "h", "V", "live", "tombstones", "guards", "slots_rewritten",
-                 "windows_rewritten", "top_level", "pending", "resizes", "resizes_last"]
+                 "windows_rewritten", "top_level", "pending", "resizes", "resizes_last", "row_begin", "rows"]
         return {n: int(out[i]) for i, n in enumerate(names)}
 
     def dump(self):
@@ -174,7 +177,7 @@ class Oracle:
         return k, v
 
     def row_offset(self):
-        out = np.zeros(self.V + 1, np.uint64)
+        out = np.zeros(self.nr + 1, np.uint64)
         lib().orc_row_offset(self._h, _p(out))
         return out
 
@@ -205,7 +208,7 @@ class Oracle:
 
     def export_csr(self):
         nnz = int(lib().orc_export_csr(self._h, None, None, None))
-        rp = np.zeros(self.V + 1, np.uint64)
+        rp = np.zeros(self.nr + 1, np.uint64)
         col = np.zeros(max(nnz, 1), np.uint32)
         val = np.zeros(max(nnz, 1), np.uint32)
         lib().orc_export_csr(self._h, _p(rp), _p(col), _p(val))

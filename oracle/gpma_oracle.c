@@ -41,6 +41,7 @@ typedef struct { uint32_t level; uint64_t seg_start_slot; uint64_t offset; uint3
 
 typedef struct orc {
   uint32_t V;
+  uint32_t rb, nr;     /* owned rows [rb, rb+nr) of a source-range shard (R24); nr = V unsharded */
   uint64_t cap;        /* slots, a power of two                       */
   uint32_t L;          /* leaf segment size (R3)                      */
   uint32_t h;          /* height: cap = L * 2^h                       */
@@ -48,7 +49,7 @@ typedef struct orc {
   uint32_t rho0, rhoh, tau0, tauh, init_bp; /* basis points (R4, R15)  */
   uint64_t *key;
   uint32_t *val;
-  uint64_t *row_offset; /* V+1 (R8)                                   */
+  uint64_t *row_offset; /* nr+1 (R8), indexed by src - rb               */
   uint64_t *tmin, *tmax;/* h+1 integer entry bounds (R5)              */
   /* last-batch diagnostics */
   trace_t *trace; uint64_t ntrace, trace_cap;
@@ -118,7 +119,7 @@ static void redispatch(orc_t *o, uint64_t l0, uint64_t nl, const uint64_t *k, co
         o->key[s] = k[lo + p];
         o->val[s] = v[lo + p];
         if (is_guard(k[lo + p]) && o->row_offset)
-          o->row_offset[(k[lo + p] >> 32) + 1] = s;
+          o->row_offset[(k[lo + p] >> 32) - o->rb + 1] = s;
       } else {
         o->key[s] = ORC_KEY_NONE;
         o->val[s] = 0;
@@ -143,7 +144,7 @@ static void trace_push(orc_t *o, uint32_t level, uint64_t start, uint64_t off, u
 static orc_t *alloc_orc(uint32_t V, int mode) {
   orc_t *o = (orc_t *)calloc(1, sizeof(orc_t));
   if (!o) return NULL;
-  o->V = V; o->mode = mode;
+  o->V = V; o->mode = mode; o->rb = 0; o->nr = V;
   o->rho0 = 800; o->rhoh = 4000; o->tau0 = 9200; o->tauh = 8000; o->init_bp = 6000;
   return o;
 }
@@ -162,13 +163,14 @@ static int cmp_kv(const void *a, const void *b) {
 
 /* Validation (SURVEY §8(b) "Errors"): RESERVED (guard column / tombstone value)
  * takes precedence over RANGE (src or dst >= V); nothing is mutated on error. */
-static int validate(uint32_t V, const uint64_t *k, const uint32_t *v, uint64_t n, int check_vals) {
+static int validate(uint32_t V, uint32_t rb, uint32_t nr, const uint64_t *k, const uint32_t *v, uint64_t n,
+                    int check_vals) {
   uint64_t i; int range = 0;
   for (i = 0; i < n; i++) {
     uint32_t src = (uint32_t)(k[i] >> 32), dst = (uint32_t)k[i];
     if (dst == ORC_GUARD_COL) return ORC_RESERVED;
     if (check_vals && v && v[i] == ORC_TOMB) return ORC_RESERVED;
-    if (src >= V || dst >= V) range = 1;
+    if (src < rb || src - rb >= nr || dst >= V) range = 1;
   }
   return range ? ORC_RANGE : ORC_OK;
 }
@@ -187,21 +189,26 @@ static uint64_t sort_unique_last(const uint64_t *k, const uint32_t *v, uint64_t 
 
 /* R15: initial capacity = smallest power of two >= 8 with E0 + V <= floor(cap * 0.6);
  * L from cap0 (R3); bump cap0 to 2L if smaller; proportional split over all leaves. */
-orc_t *orc_create(uint32_t V, const uint64_t *keys, const uint32_t *vals, uint64_t n,
-                  uint32_t leaf_slots, uint64_t cap_override, int mode, int *status) {
+/* Source-range shard (R24): the store holds rows [row_begin, row_end) -- their guards,
+ * row offsets and edges; row_end == 0 means all rows. */
+orc_t *orc_create_shard(uint32_t V, uint32_t row_begin, uint32_t row_end, const uint64_t *keys,
+                        const uint32_t *vals, uint64_t n, uint32_t leaf_slots, uint64_t cap_override,
+                        int mode, int *status) {
   kv_t *u = NULL; uint64_t m, E, i, j, cap;
   uint64_t *ek; uint32_t *ev;
   orc_t *o;
-  int st = validate(V, keys, vals, n, 1);
+  uint32_t rb = row_end > row_begin ? row_begin : 0, nr = row_end > row_begin ? row_end - row_begin : V;
+  int st = validate(V, rb, nr, keys, vals, n, 1);
   if (st) { *status = st; return NULL; }
   o = alloc_orc(V, mode);
+  o->rb = rb; o->nr = nr;
   m = sort_unique_last(keys, vals, n, &u);
-  E = m + V;
-  /* merge the sorted edges with the V guards (u<<32 | inf), R1 */
+  E = m + nr;
+  /* merge the sorted edges with the guards (u<<32 | inf) of the owned rows, R1 */
   ek = (uint64_t *)malloc(sizeof(uint64_t) * (E ? E : 1));
   ev = (uint32_t *)malloc(sizeof(uint32_t) * (E ? E : 1));
-  for (i = 0, j = 0; i < m || j < V;) {
-    uint64_t g = j < V ? (((uint64_t)j << 32) | ORC_GUARD_COL) : ORC_KEY_NONE;
+  for (i = 0, j = 0; i < m || j < nr;) {
+    uint64_t g = j < nr ? (((uint64_t)(j + rb) << 32) | ORC_GUARD_COL) : ORC_KEY_NONE;
     if (i < m && u[i].key < g) { ek[i + j] = u[i].key; ev[i + j] = u[i].val; i++; }
     else { ek[i + j] = g; ev[i + j] = 0; j++; }
   }
@@ -217,12 +224,17 @@ orc_t *orc_create(uint32_t V, const uint64_t *keys, const uint32_t *vals, uint64
   }
   o->key = (uint64_t *)malloc(sizeof(uint64_t) * cap);
   o->val = (uint32_t *)malloc(sizeof(uint32_t) * cap);
-  o->row_offset = (uint64_t *)calloc((uint64_t)V + 1, sizeof(uint64_t));
+  o->row_offset = (uint64_t *)calloc((uint64_t)nr + 1, sizeof(uint64_t));
   set_geometry(o, cap);
   redispatch(o, 0, cap / o->L, ek, ev, E);
   free(ek); free(ev);
   *status = ORC_OK;
   return o;
+}
+
+orc_t *orc_create(uint32_t V, const uint64_t *keys, const uint32_t *vals, uint64_t n,
+                  uint32_t leaf_slots, uint64_t cap_override, int mode, int *status) {
+  return orc_create_shard(V, 0, 0, keys, vals, n, leaf_slots, cap_override, mode, status);
 }
 
 /* Test hook: load a raw layout (e.g. the Fig. 3 PMA), no guards required. */
@@ -417,7 +429,7 @@ int orc_update(orc_t *o, const uint64_t *keys, const uint32_t *vals, uint64_t n,
   int st;
   if (op != ORC_INSERT && op != ORC_DELETE) return ORC_INVALID;
   if (op == ORC_INSERT && n && !vals) return ORC_INVALID;
-  st = validate(o->V, keys, vals, n, op == ORC_INSERT);
+  st = validate(o->V, o->rb, o->nr, keys, vals, n, op == ORC_INSERT);
   if (st) return st;
   o->ntrace = 0; o->slots_rewritten = 0; o->windows_rewritten = 0; o->top_level = 0;
   o->resizes_last = 0; o->pending_after_prepass = 0;
@@ -455,7 +467,7 @@ void orc_dump(const orc_t *o, uint64_t *k, uint32_t *v) {
   memcpy(v, o->val, sizeof(uint32_t) * o->cap);
 }
 void orc_row_offset(const orc_t *o, uint64_t *out) {
-  memcpy(out, o->row_offset, sizeof(uint64_t) * ((uint64_t)o->V + 1));
+  memcpy(out, o->row_offset, sizeof(uint64_t) * ((uint64_t)o->nr + 1));
 }
 void orc_level_bounds(const orc_t *o, uint64_t *mn, uint64_t *mx) {
   memcpy(mn, o->tmin, sizeof(uint64_t) * (o->h + 1));
@@ -476,6 +488,8 @@ void orc_stats(const orc_t *o, uint64_t *out) {
   out[6] = guards; out[7] = o->slots_rewritten; out[8] = o->windows_rewritten;
   out[9] = o->top_level; out[10] = o->pending_after_prepass; out[11] = o->resizes;
   out[12] = o->resizes_last;
+  out[13] = o->rb;
+  out[14] = o->nr;
 }
 /* Per-level trace of the last batch (Fig. 6 "Update Segments / Offsets / Successful
  * Flag"): records (level, seg_start_slot, offset, flag); flag 2 closes a level and
@@ -493,16 +507,17 @@ uint64_t orc_trace(const orc_t *o, uint64_t *out4, uint64_t max_records) {
 
 /* ---------------------------------------------------------------- export + analytics */
 /* CSR view of the store (Fig. 5): live edges in slot order (= key order). */
+/* rows [rb, rb+nr) of the shard (all rows unsharded): row_ptr has nr+1 entries */
 uint64_t orc_export_csr(const orc_t *o, uint64_t *row_ptr, uint32_t *col, uint32_t *val) {
   uint64_t s, nnz = 0, u;
-  if (row_ptr) for (u = 0; u <= o->V; u++) row_ptr[u] = 0;
+  if (row_ptr) for (u = 0; u <= o->nr; u++) row_ptr[u] = 0;
   for (s = 0; s < o->cap; s++) {
     if (!is_live(o, s) || is_guard(o->key[s])) continue;
     if (col) { col[nnz] = (uint32_t)o->key[s]; val[nnz] = o->val[s]; }
-    if (row_ptr) row_ptr[(o->key[s] >> 32) + 1]++;
+    if (row_ptr) row_ptr[(o->key[s] >> 32) - o->rb + 1]++;
     nnz++;
   }
-  if (row_ptr) for (u = 0; u < o->V; u++) row_ptr[u + 1] += row_ptr[u];
+  if (row_ptr) for (u = 0; u < o->nr; u++) row_ptr[u + 1] += row_ptr[u];
   return nnz;
 }
 

@@ -72,7 +72,7 @@ __device__ __forceinline__ uint32_t upper_bound_u64(const uint64_t *__restrict__
 // slots; the thread's first run is aggregated across the warp (hub rows span many lanes).
 __global__ void __launch_bounds__(TA) k_deg_count(const uint64_t *__restrict__ key,
                                                   const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
-                                                  uint32_t *deg) {
+                                                  uint32_t *deg, uint32_t rb) {
   const int lane = threadIdx.x & 31;
   const uint64_t n4 = cap / 4, n4r = (n4 + 31) & ~31ull;
   for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4r;
@@ -85,7 +85,7 @@ __global__ void __launch_bounds__(TA) k_deg_count(const uint64_t *__restrict__ k
 #pragma unroll
       for (int j = 0; j < 4; ++j) {
         if (!edge4(sl, j)) continue;
-        uint32_t u = (uint32_t)(sl.k[j] >> 32);
+        uint32_t u = (uint32_t)(sl.k[j] >> 32) - rb;   // local row
         if (u == cur) { ++c; continue; }
         if (c) {
           if (in_first) { first_src = cur; first_cnt = c; in_first = false; }
@@ -106,8 +106,8 @@ __global__ void __launch_bounds__(TA) k_deg_count(const uint64_t *__restrict__ k
 }
 
 gpma_status recompute_degrees(gpma *g, cudaStream_t s) {
-  GP_CHECK(g, cudaMemsetAsync(g->deg, 0, (uint64_t)g->V * 4, s));
-  GP_LAUNCH(g, k_deg_count, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, g->deg);
+  GP_CHECK(g, cudaMemsetAsync(g->deg, 0, (uint64_t)g->nr * 4, s));
+  GP_LAUNCH(g, k_deg_count, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, g->deg, g->rb);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
@@ -160,11 +160,12 @@ __global__ void k_bfs_list(const uint32_t *__restrict__ bm, uint32_t nwords, uin
 }
 
 __global__ void k_bfs_rowlen(const uint32_t *__restrict__ frontier, uint32_t F,
-                             const uint64_t *__restrict__ row_offset, uint64_t *__restrict__ len) {
+                             const uint64_t *__restrict__ row_offset, uint32_t rb, uint32_t nr,
+                             uint64_t *__restrict__ len) {
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < F;
        i += (uint64_t)gridDim.x * blockDim.x) {
-    uint32_t u = frontier[i];
-    len[i] = row_offset[u + 1] - row_offset[u];
+    uint32_t u = frontier[i] - rb;                  // rows outside the shard are empty here
+    len[i] = u < nr ? row_offset[u + 1] - row_offset[u] : 0;
   }
 }
 
@@ -176,7 +177,7 @@ __global__ void __launch_bounds__(TA) k_bfs_expand(const uint32_t *__restrict__ 
                                                    const uint64_t *__restrict__ row_offset,
                                                    const uint64_t *__restrict__ key,
                                                    const uint32_t *__restrict__ tmask, uint32_t L,
-                                                   int32_t *levels, int32_t depth) {
+                                                   int32_t *levels, int32_t depth, uint32_t rb) {
   const int lane = threadIdx.x & 31;
   const uint64_t total = off[F];
   const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
@@ -192,7 +193,7 @@ __global__ void __launch_bounds__(TA) k_bfs_expand(const uint32_t *__restrict__ 
     uint32_t i = i0;
     if (gi < end) {
       while (off[i + 1] <= gi) ++i;
-      uint32_t u = frontier[i];
+      uint32_t u = frontier[i] - rb;
       uint64_t s = row_offset[u] + (gi - off[i]);
       uint64_t k;
       if (edge_at(key, tmask, L, s, &k)) {
@@ -253,7 +254,16 @@ __global__ void __launch_bounds__(TA) k_bfs_sweep(const uint64_t *__restrict__ k
 
 constexpr uint32_t BFS_SPARSE_F = 4096;   // frontiers up to this size use row expansion
 
-gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
+gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
+  GP_LAUNCH(g, k_bfs_init, grid_for(g->V), TA, 0, s, levels, g->V, root);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+// One BFS level: the frontier is {v : levels[v] == depth-1} (levels may be replicated across
+// shards); the owned rows of the frontier are expanded and newly reached vertices get
+// `depth`.  *frontier = the frontier size (0: the traversal is over, nothing expanded).
+gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontier, cudaStream_t s) {
   const uint64_t V = g->V, nl = g->cap / g->L;
   GP_CHECK(g, ensure(g->b_an[0], (V + 1) * 4, s));
   GP_CHECK(g, ensure(g->b_an[2], (std::max<uint64_t>(V, nl) + 2) * 8, s));
@@ -267,31 +277,39 @@ gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
   uint32_t *bm = (uint32_t *)g->b_an[3].p;
   uint32_t *F_d = reinterpret_cast<uint32_t *>(&g->ctrl_d->sum);
   const uint32_t *tmask = tmask_of(g);
-  GP_LAUNCH(g, k_bfs_init, grid_for(V), TA, 0, s, levels, (uint32_t)V, root);
-  for (int32_t depth = 1;; ++depth) {
+  GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
+  GP_LAUNCH(g, k_bfs_frontier, grid_for(V), TA, 0, s, levels, (uint32_t)V, depth - 1, bm, F_d);
+  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  const uint32_t F = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
+  *frontier = F;
+  if (!F) return GPMA_OK;
+  if (F <= BFS_SPARSE_F) {
     GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
-    GP_LAUNCH(g, k_bfs_frontier, grid_for(V), TA, 0, s, levels, (uint32_t)V, depth - 1, bm, F_d);
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
-    GP_CHECK(g, cudaStreamSynchronize(s));
-    const uint32_t F = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
-    if (!F) break;
-    if (F <= BFS_SPARSE_F) {
-      GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
-      GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, F_d);
-      GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, off);
-      scan_u64(g, off, off, F, s);
-      GP_LAUNCH(g, k_bfs_expand, MAX_RESIDENT_BLOCKS, TA, 0, s, list, F, off, g->row_offset, g->key, tmask,
-                g->L, levels, depth);
-    } else {
-      GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, act);
-      scan_u32(g, act, apos, nl, s);
-      GP_LAUNCH(g, k_bfs_leaf_list, grid_for(nl), TA, 0, s, act, apos, nl, alist);
-      GP_LAUNCH(g, k_bfs_sweep, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask, g->L, alist, apos + nl, bm,
-                levels, depth);
-    }
+    GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, F_d);
+    GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, g->rb, g->nr, off);
+    scan_u64(g, off, off, F, s);
+    GP_LAUNCH(g, k_bfs_expand, MAX_RESIDENT_BLOCKS, TA, 0, s, list, F, off, g->row_offset, g->key, tmask, g->L,
+              levels, depth, g->rb);
+  } else {
+    GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, act);
+    scan_u32(g, act, apos, nl, s);
+    GP_LAUNCH(g, k_bfs_leaf_list, grid_for(nl), TA, 0, s, act, apos, nl, alist);
+    GP_LAUNCH(g, k_bfs_sweep, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask, g->L, alist, apos + nl, bm, levels,
+              depth);
   }
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
+}
+
+gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
+  gpma_status st = bfs_init(g, root, levels, s);
+  for (int32_t depth = 1; st == GPMA_OK; ++depth) {
+    uint32_t F = 0;
+    st = bfs_level(g, levels, depth, &F, s);
+    if (!F) break;
+  }
+  return st;
 }
 
 // ------------------------------------------------------------------ CC
@@ -414,6 +432,38 @@ __global__ void k_cc_final(uint32_t *p, uint32_t *labels, uint32_t V) {
   }
 }
 
+__global__ void k_cc_changed(const uint32_t *__restrict__ a, const uint32_t *__restrict__ b, uint32_t V, Ctrl *c) {
+  uint64_t n = 0;
+  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
+       v += (uint64_t)gridDim.x * blockDim.x)
+    n += a[v] != b[v];
+  for (int o = 16; o; o >>= 1) n += __shfl_xor_sync(0xffffffffu, n, o);
+  if ((threadIdx.x & 31) == 0 && n) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)n);
+}
+
+// One hooking round over the owned edges on top of `labels` (a forest with p[x] <= x, e.g.
+// the element-wise minimum of other shards' labels): sampled round, compression, full pass,
+// full compression.  *changed = vertices whose label moved (0 on every shard = fixpoint).
+gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cudaStream_t s) {
+  const uint64_t V = g->V;
+  GP_CHECK(g, ensure(g->b_an[1], (V + 1) * 4, s));
+  uint32_t *prev = (uint32_t *)g->b_an[1].p;
+  const uint32_t *tmask = tmask_of(g);
+  if (init) GP_LAUNCH(g, k_cc_init, grid_for(V), TA, 0, s, labels, g->V);
+  GP_CHECK(g, cudaMemcpyAsync(prev, labels, V * 4, cudaMemcpyDeviceToDevice, s));
+  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
+  GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
+  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
+  GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
+  GP_CHECK(g, cudaMemsetAsync(&g->ctrl_d->sum, 0, 8, s));
+  GP_LAUNCH(g, k_cc_changed, grid_for(V), TA, 0, s, labels, prev, g->V, g->ctrl_d);
+  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, &g->ctrl_d->sum, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  *changed = g->ctrl_h->sum;
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s) {
   GP_CHECK(g, ensure(g->b_an[0], ((uint64_t)g->V + 1) * 4, s));
   uint32_t *p = (uint32_t *)g->b_an[0].p;
@@ -479,14 +529,14 @@ __global__ void k_pr_prep(T *__restrict__ x, const uint32_t *__restrict__ deg,
 // y[v] += contrib[u] over the live edges u -> v (push SpMV): two groups of 4 slots per
 // thread, all loads (keys, masks, contributions) issued before the fire-and-forget REDs.
 template <typename A>
-__device__ __forceinline__ void pr_contribs(const Slot4 &sl, const A *__restrict__ contrib, A cv[4]) {
+__device__ __forceinline__ void pr_contribs(const Slot4 &sl, const A *__restrict__ contrib, A cv[4], uint32_t rb) {
   uint32_t cu = 0xFFFFFFFFu;
   A c = 0;
 #pragma unroll
   for (int j = 0; j < 4; ++j) {
     cv[j] = 0;
     if (!edge4(sl, j)) continue;
-    uint32_t u = (uint32_t)(sl.k[j] >> 32);
+    uint32_t u = (uint32_t)(sl.k[j] >> 32) - rb;     // contributions are per owned row
     if (u != cu) { cu = u; c = __ldcs(contrib + u); }
     cv[j] = c;
   }
@@ -502,7 +552,7 @@ __device__ __forceinline__ void pr_scatter(const Slot4 &sl, const A cv[4], A *y)
 template <typename A>
 __global__ void __launch_bounds__(TA) k_pr_push(const uint64_t *__restrict__ key,
                                                 const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
-                                                const A *__restrict__ contrib, A *y) {
+                                                const A *__restrict__ contrib, A *y, uint32_t rb) {
   const uint64_t n4 = cap / 4, stride = (uint64_t)gridDim.x * blockDim.x;
   for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4; t += 2 * stride) {
     Slot4 a, b;
@@ -510,8 +560,8 @@ __global__ void __launch_bounds__(TA) k_pr_push(const uint64_t *__restrict__ key
     load4(key, tmask, L, t * 4, a);
     if (hb) load4(key, tmask, L, (t + stride) * 4, b);
     A ca[4], cb[4];
-    pr_contribs(a, contrib, ca);
-    if (hb) pr_contribs(b, contrib, cb);
+    pr_contribs(a, contrib, ca, rb);
+    if (hb) pr_contribs(b, contrib, cb, rb);
     pr_scatter(a, ca, y);
     if (hb) pr_scatter(b, cb, y);
   }
@@ -558,7 +608,8 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
   int it = 0, cur = 0;
   while (it < max_iter) {
-    GP_LAUNCH(g, k_pr_push<A>, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, contrib, y);
+    GP_LAUNCH(g, k_pr_push<A>, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, contrib, y,
+              0u);
     GP_CHECK(g, cudaMemsetAsync(acc + 2, 0, sizeof(double), s));
     GP_CHECK(g, cudaMemsetAsync(acc + (cur ^ 1), 0, sizeof(double), s));
     GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
@@ -576,6 +627,70 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   return GPMA_OK;
 }
 
+// ---- distributed PageRank primitives (replicated x, exact fixed-point partial sums)
+__global__ void k_prd_init(double *x, uint32_t V) {
+  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
+       v += (uint64_t)gridDim.x * blockDim.x)
+    x[v] = 1.0 / (double)V;
+}
+
+// contributions of the owned rows; their dangling mass (fixed point) into y[V]
+__global__ void k_prd_contrib(const double *__restrict__ x, const uint32_t *__restrict__ deg, uint32_t rb,
+                              uint32_t nr, unsigned long long *__restrict__ contrib, unsigned long long *y,
+                              uint32_t V) {
+  unsigned long long dl = 0;
+  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < nr;
+       u += (uint64_t)gridDim.x * blockDim.x) {
+    const double xv = x[u + rb];
+    const uint32_t dg = deg[u];
+    contrib[u] = dg ? PrAcc<double>::enc(xv / (double)dg) : 0ull;
+    if (!dg) dl += PrAcc<double>::enc(xv);
+  }
+  for (int o = 16; o; o >>= 1) dl += __shfl_xor_sync(0xffffffffu, dl, o);
+  if ((threadIdx.x & 31) == 0 && dl) atomicAdd(y + V, dl);
+}
+
+// x' = (1-d)/V + d (y + D/V) for every vertex (replicated), err = ||x'-x||_1, y := 0
+__global__ void k_prd_update(double *__restrict__ x, unsigned long long *__restrict__ y, uint32_t V, double d,
+                             double *err) {
+  __shared__ double red[32];
+  const double base = (1.0 - d) / (double)V + d * (PrAcc<double>::dec(y[V]) / (double)V);
+  double e = 0;
+  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
+       v += (uint64_t)gridDim.x * blockDim.x) {
+    const double nx = base + d * PrAcc<double>::dec(y[v]);
+    e += fabs(nx - x[v]);
+    x[v] = nx;
+    y[v] = 0;
+  }
+  double se = block_sum_d(e, red);
+  if (threadIdx.x == 0 && se != 0) atomicAdd(err, se);
+}
+
+gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
+  GP_CHECK(g, ensure(g->b_an[1], ((uint64_t)g->nr + 1) * 8, s));
+  unsigned long long *contrib = (unsigned long long *)g->b_an[1].p;
+  unsigned long long *yy = (unsigned long long *)y;
+  if (init) GP_LAUNCH(g, k_prd_init, grid_for(g->V), TA, 0, s, x, g->V);
+  GP_LAUNCH(g, k_prd_contrib, grid_for(g->nr), TA, 0, s, x, g->deg, g->rb, g->nr, contrib, yy, g->V);
+  GP_LAUNCH(g, k_pr_push<unsigned long long>, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap,
+            contrib, yy, g->rb);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+gpma_status pr_update(gpma *g, double *x, uint64_t *y, double d, double *err, cudaStream_t s) {
+  double *e_d = reinterpret_cast<double *>(&g->ctrl_d->sum2);
+  GP_CHECK(g, cudaMemsetAsync(e_d, 0, 8, s));
+  GP_LAUNCH(g, k_prd_update, grid_for(g->V), TA, 0, s, x, (unsigned long long *)y, g->V, d, e_d);
+  GP_CHECK(g, cudaMemsetAsync(y + g->V, 0, 8, s));
+  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, e_d, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  memcpy(err, &g->ctrl_h->sum2, 8);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 gpma_status pagerank_f64(gpma *g, double *x, int warm, double d, double tol, int max_iter, int *iters,
                          cudaStream_t s) {
   return pagerank_t<double>(g, x, warm, d, tol, max_iter, iters, s);
@@ -589,11 +704,11 @@ gpma_status pagerank_f32(gpma *g, float *x, int warm, float d, float tol, int ma
 // ------------------------------------------------------------------ export CSR
 // guards per leaf from the row offsets (R8: row_offset[u+1] = slot of guard u)
 __global__ void k_exp_guards(const uint64_t *__restrict__ row_offset, const uint64_t *__restrict__ key,
-                             uint32_t V, uint32_t L, uint32_t *__restrict__ gl) {
-  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < V;
+                             uint32_t rb, uint32_t nr, uint32_t L, uint32_t *__restrict__ gl) {
+  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < nr;
        u += (uint64_t)gridDim.x * blockDim.x) {
     uint64_t s = row_offset[u + 1];
-    if (key[s] == ((u << 32) | COL_GUARD)) atomicAdd(&gl[s / L], 1u);
+    if (key[s] == (((u + rb) << 32) | COL_GUARD)) atomicAdd(&gl[s / L], 1u);
   }
 }
 
@@ -612,7 +727,7 @@ __global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ k
                                                   const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
                                                   const uint64_t *__restrict__ lbase,
                                                   uint64_t *__restrict__ row_ptr, uint32_t *__restrict__ col,
-                                                  uint32_t *__restrict__ cval) {
+                                                  uint32_t *__restrict__ cval, uint32_t rb) {
   const int lane = threadIdx.x & 31;
   const uint32_t lpl = L / 4;                    // lanes per leaf (1..8)
   const uint64_t n4 = cap / 4, n4r = (n4 + 31) & ~31ull;
@@ -642,7 +757,7 @@ __global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ k
         cval[r] = vs[j];
         ++r;
       } else if (is_guard_key(sl.k[j])) {
-        row_ptr[(sl.k[j] >> 32) + 1] = r;
+        row_ptr[(sl.k[j] >> 32) - rb + 1] = r;
       }
     }
   }
@@ -656,7 +771,7 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
   uint64_t *lc = (uint64_t *)g->b_lpre.p;
   uint32_t *gl = (uint32_t *)g->b_an[0].p;
   GP_CHECK(g, cudaMemsetAsync(gl, 0, nl * 4, s));
-  GP_LAUNCH(g, k_exp_guards, grid_for(g->V), TA, 0, s, g->row_offset, g->key, g->V, g->L, gl);
+  GP_LAUNCH(g, k_exp_guards, grid_for(g->nr), TA, 0, s, g->row_offset, g->key, g->rb, g->nr, g->L, gl);
   GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gl, nl, lc);
   scan_u64(g, lc, lc, nl, s);
   GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, lc + nl, 8, cudaMemcpyDeviceToHost, s));
@@ -670,7 +785,7 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
   }
   GP_CHECK(g, cudaMemsetAsync(row_ptr, 0, 8, s));
   GP_LAUNCH(g, k_exp_write, grid_for(g->cap / 4), TA, 0, s, g->key, g->val, tmask_of(g), g->L, g->cap, lc,
-            row_ptr, col, val);
+            row_ptr, col, val, g->rb);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }

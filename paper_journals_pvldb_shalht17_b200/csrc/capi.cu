@@ -90,6 +90,14 @@ gpma_status apply_config(gpma *g, const gpma_config *cfg, uint32_t *leaf, uint64
   g->tauh = c.tau_root_bp;
   g->init_bp = c.init_density_bp;
   g->mode = c.delete_mode;
+  if (c.row_end > c.row_begin) {
+    if (c.row_end > g->V) return GPMA_ERR_INVALID_ARG;
+    g->rb = c.row_begin;
+    g->nr = c.row_end - c.row_begin;
+  } else {
+    g->rb = 0;
+    g->nr = g->V;
+  }
   *leaf = c.leaf_slots;
   *cap = c.initial_capacity;
   return GPMA_OK;
@@ -206,14 +214,14 @@ gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t l
     uint64_t nl = capacity / leaf_slots;
     if (cudaMallocAsync((void **)&g->key, capacity * 8, s) || cudaMallocAsync((void **)&g->val, capacity * 4, s) ||
         cudaMallocAsync((void **)&g->cnt, nl * 8, s) || cudaMallocAsync((void **)&g->head, nl * 8, s) ||
-        cudaMallocAsync((void **)&g->row_offset, ((uint64_t)num_vertices + 1) * 8, s) ||
-        cudaMallocAsync((void **)&g->deg, (uint64_t)num_vertices * 4, s)) {
+        cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s) ||
+        cudaMallocAsync((void **)&g->deg, (uint64_t)g->nr * 4 + 4, s)) {
       cudaGetLastError();
       st = GPMA_ERR_OOM;
     }
   }
   if (st == GPMA_OK) {
-    cudaMemsetAsync(g->row_offset, 0, ((uint64_t)num_vertices + 1) * 8, s);
+    cudaMemsetAsync(g->row_offset, 0, ((uint64_t)g->nr + 1) * 8, s);
     st = gp::load_raw(g, keys, vals, s);
   }
   if (st == GPMA_OK && cudaStreamSynchronize(s) != cudaSuccess) st = GPMA_ERR_CUDA;
@@ -276,6 +284,7 @@ gpma_status gpma_pagerank(gpma_t *g, double *rank, int warm_start, double dampin
   gpma_status st = begin(g);
   if (st) return st;
   if (!rank || max_iter < 0 || !(damping >= 0.0 && damping <= 1.0) || !(tol_l1 >= 0.0)) return GPMA_ERR_INVALID_ARG;
+  if (g->nr != g->V) return GPMA_ERR_INVALID_ARG;   // sharded: use gpma_pr_push / gpma_pr_update
   cudaStream_t s = (cudaStream_t)stream;
   Out o(g, rank, (size_t)g->V * 8, s);
   void *d;
@@ -291,6 +300,7 @@ gpma_status gpma_pagerank_f32(gpma_t *g, float *rank, int warm_start, float damp
   gpma_status st = begin(g);
   if (st) return st;
   if (!rank || max_iter < 0 || !(damping >= 0.0f && damping <= 1.0f) || !(tol_l1 >= 0.0f)) return GPMA_ERR_INVALID_ARG;
+  if (g->nr != g->V) return GPMA_ERR_INVALID_ARG;
   cudaStream_t s = (cudaStream_t)stream;
   Out o(g, rank, (size_t)g->V * 4, s);
   void *d;
@@ -313,7 +323,7 @@ gpma_status gpma_export_csr(gpma_t *g, uint64_t *row_ptr, uint32_t *col, uint32_
     if (nnz_out) *nnz_out = nnz;
     return end(g, st);
   }
-  Out orp(g, row_ptr, ((size_t)g->V + 1) * 8, s), oc(g, col, (size_t)nnz_capacity * 4, s),
+  Out orp(g, row_ptr, ((size_t)g->nr + 1) * 8, s), oc(g, col, (size_t)nnz_capacity * 4, s),
       ov(g, val, (size_t)nnz_capacity * 4, s);
   void *drp, *dc, *dv;
   if (cudaError_t e = orp.dev(&drp, false)) return gp::cuda_fail(g, e, "export staging");
@@ -352,7 +362,7 @@ gpma_status gpma_debug_dump(gpma_t *g, uint64_t *keys, uint32_t *vals, uint64_t 
   cudaStream_t s = (cudaStream_t)stream;
   uint64_t nl = g->cap / g->L;
   struct { void *dst; const void *src; size_t bytes; } cp[] = {
-      {keys, g->key, g->cap * 8}, {vals, g->val, g->cap * 4}, {row_offset, g->row_offset, ((size_t)g->V + 1) * 8},
+      {keys, g->key, g->cap * 8}, {vals, g->val, g->cap * 4}, {row_offset, g->row_offset, ((size_t)g->nr + 1) * 8},
       {leaf_live, g->cnt, nl * 4}, {heads, g->head, nl * 8}};
   for (auto &c : cp)
     if (c.dst)
@@ -411,6 +421,53 @@ gpma_status gpma_debug_profile_read(gpma_t *g, char *buf, size_t buflen) {
   g->prof_recs.clear();
   g->ev_used = 0;
   return GPMA_OK;
+}
+
+// ---- sharded-store primitives (device pointers)
+gpma_status gpma_route(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, uint32_t nranks,
+                       uint64_t *out_keys, uint32_t *out_vals, uint64_t *counts, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if ((n && (!keys || !out_keys || !out_vals)) || !counts || nranks == 0 || nranks > 256)
+    return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::route(g, keys, vals, n, nranks, out_keys, out_vals, counts, (cudaStream_t)stream));
+}
+
+gpma_status gpma_bfs_init(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!levels || root >= g->V) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::bfs_init(g, root, levels, (cudaStream_t)stream));
+}
+
+gpma_status gpma_bfs_level(gpma_t *g, int32_t *levels, int32_t depth, uint32_t *frontier_size,
+                           gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!levels || !frontier_size || depth < 1) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::bfs_level(g, levels, depth, frontier_size, (cudaStream_t)stream));
+}
+
+gpma_status gpma_cc_round(gpma_t *g, uint32_t *labels, int init, uint64_t *changed, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!labels || !changed) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::cc_round(g, labels, init, changed, (cudaStream_t)stream));
+}
+
+gpma_status gpma_pr_push(gpma_t *g, double *x, int init, uint64_t *y, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!x || !y) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::pr_push(g, x, init, y, (cudaStream_t)stream));
+}
+
+gpma_status gpma_pr_update(gpma_t *g, double *x, uint64_t *y, double damping, double *err,
+                           gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!x || !y || !err || !(damping >= 0.0 && damping <= 1.0)) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::pr_update(g, x, y, damping, err, (cudaStream_t)stream));
 }
 
 uint64_t gpma_kernel_launches(const gpma_t *g) { return g ? g->launches : 0; }

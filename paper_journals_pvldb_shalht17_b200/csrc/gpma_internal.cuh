@@ -57,6 +57,7 @@ struct LevelBufs {
 struct gpma {
   // geometry (R3, R4, R5, R15)
   uint32_t V = 0, L = 0, h = 0, mode = 0;
+  uint32_t rb = 0, nr = 0;        // owned rows [rb, rb + nr) (shard, R24); nr = V unsharded
   uint64_t cap = 0;
   uint32_t rho0 = 800, rhoh = 4000, tau0 = 9200, tauh = 8000, init_bp = 6000;
   std::vector<uint64_t> tmin, tmax;
@@ -129,6 +130,17 @@ void scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream
 // the index (0/1) of the buffer pair holding the result.
 int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1, uint64_t n,
                      const int *shifts, int nshift, cudaStream_t s);
+gpma_status radix_partition_owner(gpma *g, const uint64_t *k0, const uint32_t *v0, uint64_t *k1, uint32_t *v1,
+                                  uint64_t n, uint32_t div, uint32_t nranks, uint64_t *starts_dev,
+                                  cudaStream_t s);
+// distributed primitives (dist.cu / analytics.cu)
+gpma_status route(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, uint32_t nranks,
+                  uint64_t *out_keys, uint32_t *out_vals, uint64_t *counts_host, cudaStream_t s);
+gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s);
+gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontier, cudaStream_t s);
+gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cudaStream_t s);
+gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s);
+gpma_status pr_update(gpma *g, double *x, uint64_t *y, double d, double *err, cudaStream_t s);
 // digit shifts covering the significant bits of keys with src, dst < V
 int key_shifts(uint32_t V, int *shifts);
 

@@ -231,10 +231,15 @@ constexpr int RS_ITEMS = 8;
 constexpr int RS_WARPS = RS_THREADS / 32;
 constexpr int RS_TILE = RS_THREADS * RS_ITEMS;
 
+// digit of a key: 8 key bits at `shift`, or (div != 0) the owner rank src / div (routing)
+__device__ __forceinline__ uint32_t rdigit(uint64_t k, int shift, uint32_t div) {
+  return div ? min(255u, (uint32_t)(k >> 32) / div) : (uint32_t)(k >> shift) & 255u;
+}
+
 __global__ void __launch_bounds__(RS_THREADS) k_radix_hist(const uint64_t *__restrict__ keys,
                                                            uint64_t n, int shift,
                                                            uint32_t *__restrict__ hist,
-                                                           uint32_t ntiles) {
+                                                           uint32_t ntiles, uint32_t div) {
   __shared__ uint32_t h[256];
   h[threadIdx.x] = 0;
   __syncthreads();
@@ -242,7 +247,7 @@ __global__ void __launch_bounds__(RS_THREADS) k_radix_hist(const uint64_t *__res
 #pragma unroll 4
   for (int j = 0; j < RS_ITEMS; ++j) {
     uint64_t i = base + (uint64_t)j * RS_THREADS + threadIdx.x;
-    if (i < n) atomicAdd(&h[(keys[i] >> shift) & 255u], 1u);
+    if (i < n) atomicAdd(&h[rdigit(keys[i], shift, div)], 1u);
   }
   __syncthreads();
   hist[(uint64_t)threadIdx.x * ntiles + blockIdx.x] = h[threadIdx.x];
@@ -251,7 +256,7 @@ __global__ void __launch_bounds__(RS_THREADS) k_radix_hist(const uint64_t *__res
 __global__ void __launch_bounds__(RS_THREADS) k_radix_scatter(
     const uint64_t *__restrict__ kin, const uint32_t *__restrict__ vin, uint64_t *__restrict__ kout,
     uint32_t *__restrict__ vout, uint64_t n, int shift, const uint32_t *__restrict__ hscan,
-    uint32_t ntiles) {
+    uint32_t ntiles, uint32_t div) {
   __shared__ uint32_t wc[RS_WARPS][256];
   for (int d = threadIdx.x; d < RS_WARPS * 256; d += RS_THREADS) (&wc[0][0])[d] = 0;
   __syncthreads();
@@ -271,7 +276,7 @@ __global__ void __launch_bounds__(RS_THREADS) k_radix_scatter(
   for (int j = 0; j < RS_ITEMS; ++j) {
     uint64_t i = base + j * 32 + lane;
     bool ok = i < n;
-    uint32_t d = ok ? (uint32_t)(k[j] >> shift) & 255u : 256u + lane;
+    uint32_t d = ok ? rdigit(k[j], shift, div) : 256u + lane;
     uint32_t peers = __match_any_sync(0xffffffffu, d);
     uint32_t cur = ok ? wc[w][d] : 0u;
     __syncwarp();
@@ -296,7 +301,7 @@ __global__ void __launch_bounds__(RS_THREADS) k_radix_scatter(
   for (int j = 0; j < RS_ITEMS; ++j) {
     uint64_t i = base + j * 32 + lane;
     if (i < n) {
-      uint32_t d = (uint32_t)(k[j] >> shift) & 255u;
+      uint32_t d = rdigit(k[j], shift, div);
       uint64_t pos = (uint64_t)hscan[(uint64_t)d * ntiles + blockIdx.x] + wc[w][d] + r[j];
       kout[pos] = k[j];
       vout[pos] = v[j];
@@ -315,13 +320,35 @@ int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t
   uint32_t *vs[2] = {v0, v1};
   int cur = 0;
   for (int p = 0; p < nshift; ++p) {
-    GP_LAUNCH(g, k_radix_hist, ntiles, RS_THREADS, 0, s, ks[cur], n, shifts[p], hist, ntiles);
+    GP_LAUNCH(g, k_radix_hist, ntiles, RS_THREADS, 0, s, ks[cur], n, shifts[p], hist, ntiles, 0u);
     scan_u32(g, hist, hist, hn, s);
     GP_LAUNCH(g, k_radix_scatter, ntiles, RS_THREADS, 0, s, ks[cur], vs[cur], ks[cur ^ 1],
-              vs[cur ^ 1], n, shifts[p], hist, ntiles);
+              vs[cur ^ 1], n, shifts[p], hist, ntiles, 0u);
     cur ^= 1;
   }
   return cur;
+}
+
+__global__ void k_owner_starts(const uint32_t *__restrict__ hscan, uint32_t ntiles, uint32_t nranks,
+                               uint64_t n, uint64_t *__restrict__ starts) {
+  for (uint32_t d = threadIdx.x; d <= nranks; d += blockDim.x)
+    starts[d] = d < nranks ? hscan[(uint64_t)d * ntiles] : n;
+}
+
+// One stable counting pass by owner = src / div (the routing step of the sharded store).
+gpma_status radix_partition_owner(gpma *g, const uint64_t *k0, const uint32_t *v0, uint64_t *k1, uint32_t *v1,
+                                  uint64_t n, uint32_t div, uint32_t nranks, uint64_t *starts_dev,
+                                  cudaStream_t s) {
+  const uint32_t ntiles = (uint32_t)std::max<uint64_t>(1, (n + RS_TILE - 1) / RS_TILE);
+  const uint64_t hn = (uint64_t)ntiles * 256;
+  GP_CHECK(g, ensure(g->b_hist, (hn + 1) * sizeof(uint32_t), s));
+  uint32_t *hist = (uint32_t *)g->b_hist.p;
+  GP_LAUNCH(g, k_radix_hist, ntiles, RS_THREADS, 0, s, k0, n, 0, hist, ntiles, div);
+  scan_u32(g, hist, hist, hn, s);
+  GP_LAUNCH(g, k_radix_scatter, ntiles, RS_THREADS, 0, s, k0, v0, k1, v1, n, 0, hist, ntiles, div);
+  GP_LAUNCH(g, k_owner_starts, 1, 256, 0, s, hist, ntiles, nranks, n, starts_dev);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
 }
 
 }  // namespace gp

@@ -37,7 +37,7 @@ __device__ __forceinline__ uint32_t locate_leaf(const uint64_t *__restrict__ hea
 
 // ------------------------------------------------------------------ validate
 __global__ void k_validate(const uint64_t *__restrict__ keys, const uint32_t *__restrict__ vals,
-                           uint64_t n, uint32_t V, int check_vals, Ctrl *c) {
+                           uint64_t n, uint32_t V, uint32_t rb, uint32_t nr, int check_vals, Ctrl *c) {
   uint32_t e = 0;
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
        i += (uint64_t)gridDim.x * blockDim.x) {
@@ -45,7 +45,7 @@ __global__ void k_validate(const uint64_t *__restrict__ keys, const uint32_t *__
     uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
     if (dst == COL_GUARD) e |= 2u;
     if (check_vals && vals[i] == VAL_TOMB) e |= 2u;
-    if (src >= V || dst >= V) e |= 1u;
+    if (src - rb >= nr || dst >= V) e |= 1u;    // src outside the owned rows (wraps)
   }
   e = __reduce_or_sync(0xffffffffu, e);
   if (e && (threadIdx.x & 31) == 0) atomicOr(&c->err, e);
@@ -58,7 +58,7 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
                           uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
                           uint32_t nleaves, uint32_t L, int op, int mode,
                           uint32_t *__restrict__ keep, uint32_t *__restrict__ tgt, Ctrl *c,
-                          uint32_t *__restrict__ tmask, uint32_t *__restrict__ deg) {
+                          uint32_t *__restrict__ tmask, uint32_t *__restrict__ deg, uint32_t rb) {
   uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
   uint32_t uniq = 0;
   if (i < n) {
@@ -73,7 +73,7 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
         if (x == k) { hit = base + p; break; }
         if (x == KEY_NONE || x > k) break;
       }
-      const uint32_t src = (uint32_t)(k >> 32);
+      const uint32_t src = (uint32_t)(k >> 32) - rb;   // local row
       const uint32_t bit = hit != KEY_NONE ? 1u << (uint32_t)(hit - base) : 0u;
       if (op == GPMA_INSERT) {
         if (hit != KEY_NONE) {                      // overwrite (R11) or revive (R12)
@@ -140,6 +140,7 @@ struct Lvl {
   uint64_t tmin, tmax;
   int op;
   int force;           // resize: accept the single root window unconditionally
+  uint32_t rb;         // first owned row (row offsets are local)
 };
 
 __global__ void k_lvl_flags(Lvl a) {
@@ -339,7 +340,7 @@ __global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *
       uint64_t k = a.wk[e];
       key[s] = k;
       val[s] = a.wv[e];
-      if (is_guard_key(k)) row_offset[(k >> 32) + 1] = s;
+      if (is_guard_key(k)) row_offset[(k >> 32) - a.rb + 1] = s;
     } else {
       key[s] = KEY_NONE;
       val[s] = 0;
@@ -370,7 +371,7 @@ __global__ void k_lvl_summary(Lvl a, Ctrl *c) {
 __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *__restrict__ wv,
                               uint64_t N, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
                               uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset,
-                              uint32_t L, uint64_t nleaves) {
+                              uint32_t L, uint64_t nleaves, uint32_t rb) {
   uint32_t *tmask = cnt + nleaves;
   const uint64_t cap = nleaves * L;
   for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
@@ -381,7 +382,7 @@ __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *_
       uint64_t k = wk[lo + p];
       key[s] = k;
       val[s] = wv[lo + p];
-      if (is_guard_key(k)) row_offset[(k >> 32) + 1] = s;
+      if (is_guard_key(k)) row_offset[(k >> 32) - rb + 1] = s;
     } else {
       key[s] = KEY_NONE;
       val[s] = 0;
@@ -462,23 +463,22 @@ __global__ void k_count_slots(const uint64_t *__restrict__ key, const uint32_t *
 // Edge j with source u lands at j + u; guard u at (#edges with src <= u) + u.
 __global__ void k_place_edges(const uint64_t *__restrict__ sk, const uint32_t *__restrict__ sv,
                               const uint32_t *__restrict__ pos, const uint32_t *__restrict__ keep,
-                              uint64_t n, uint64_t *__restrict__ wk, uint32_t *__restrict__ wv) {
+                              uint64_t n, uint64_t *__restrict__ wk, uint32_t *__restrict__ wv, uint32_t rb) {
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
        i += (uint64_t)gridDim.x * blockDim.x) {
     if (!keep[i]) continue;
     uint64_t k = sk[i];
-    uint64_t d = (uint64_t)pos[i] + (k >> 32);
+    uint64_t d = (uint64_t)pos[i] + ((k >> 32) - rb);   // guards of the owned rows before it
     wk[d] = k;
     wv[d] = sv[i];
   }
 }
 
-__global__ void k_place_guards(const uint64_t *__restrict__ wk_edges_sorted_unused, uint32_t V,
-                               const uint64_t *__restrict__ ek, uint64_t m, uint64_t *__restrict__ wk,
-                               uint32_t *__restrict__ wv) {
-  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < V;
+__global__ void k_place_guards(uint32_t rb, uint32_t nr, const uint64_t *__restrict__ ek, uint64_t m,
+                               uint64_t *__restrict__ wk, uint32_t *__restrict__ wv) {
+  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < nr;
        u += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t gk = (u << 32) | COL_GUARD;
+    uint64_t gk = ((u + rb) << 32) | COL_GUARD;
     // number of edges with key < guard key, searched in the dense edge list ek[0..m)
     uint64_t lo = 0, hi = m;
     while (lo < hi) {
@@ -510,7 +510,7 @@ __global__ void k_compact_kv(const uint32_t *__restrict__ keep, const uint32_t *
 
 __global__ void k_raw_counts(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val,
                              uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset, uint32_t L,
-                             uint64_t nleaves, uint32_t V) {
+                             uint64_t nleaves, uint32_t rb, uint32_t nr) {
   for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
        l += (uint64_t)gridDim.x * blockDim.x) {
     uint32_t c = 0, m = 0;
@@ -520,7 +520,7 @@ __global__ void k_raw_counts(const uint64_t *__restrict__ key, const uint32_t *_
       if (k == KEY_NONE) continue;
       if (val[s] != VAL_TOMB) ++c;
       else m |= 1u << p;
-      if (is_guard_key(k) && (k >> 32) < V) row_offset[(k >> 32) + 1] = s;
+      if (is_guard_key(k) && (uint32_t)(k >> 32) - rb < nr) row_offset[(k >> 32) - rb + 1] = s;
     }
     cnt[l] = c;
     cnt[nleaves + l] = m;
@@ -587,7 +587,7 @@ gpma_status build_from_sorted(gpma *g, const uint64_t *wk, const uint32_t *wv, u
                               cudaStream_t s) {
   uint64_t nl = g->cap / g->L;
   GP_LAUNCH(g, k_layout_even, grid_for(g->cap), TB, 0, s, wk, wv, N, g->key, g->val, g->cnt,
-            g->row_offset, g->L, nl);
+            g->row_offset, g->L, nl, g->rb);
   GP_CHECK(g, cudaGetLastError());
   gpma_status st = recompute_heads(g, s);
   if (st) return st;
@@ -599,7 +599,7 @@ gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaSt
   GP_CHECK(g, cudaMemcpyAsync(g->val, vals, g->cap * 4, cudaMemcpyDefault, s));
   uint64_t nl = g->cap / g->L;
   GP_LAUNCH(g, k_raw_counts, grid_for(nl), TB, 0, s, g->key, g->val, g->cnt, g->row_offset, g->L, nl,
-            g->V);
+            g->rb, g->nr);
   GP_CHECK(g, cudaGetLastError());
   gpma_status st = recompute_heads(g, s);
   if (st) return st;
@@ -632,7 +632,8 @@ static gpma_status validate(gpma *g, const uint64_t *keys, const uint32_t *vals,
                             bool check_vals, cudaStream_t s) {
   gpma_status st = zero_ctrl(g, s);
   if (st) return st;
-  GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, keys, vals, n, g->V, check_vals ? 1 : 0, g->ctrl_d);
+  GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, keys, vals, n, g->V, g->rb, g->nr, check_vals ? 1 : 0,
+            g->ctrl_d);
   if ((st = read_ctrl(g, s))) return st;
   if (g->ctrl_h->err & 2u) return GPMA_ERR_RESERVED;
   if (g->ctrl_h->err & 1u) return GPMA_ERR_RANGE;
@@ -677,7 +678,7 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
     ek = uk;
     ev = uv;
   }
-  const uint64_t E = m + g->V;
+  const uint64_t E = m + g->nr;
   uint64_t cap;
   if (cap_override) {
     cap = cap_override;
@@ -694,9 +695,9 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
   }
   set_geometry(g, cap);
   if ((st = alloc_store(g, cap, &g->key, &g->val, &g->cnt, &g->head, s))) return st;
-  GP_CHECK(g, cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->V + 1) * 8, s));
-  GP_CHECK(g, cudaMemsetAsync(g->row_offset, 0, ((uint64_t)g->V + 1) * 8, s));
-  GP_CHECK(g, cudaMallocAsync((void **)&g->deg, (uint64_t)g->V * 4, s));
+  GP_CHECK(g, cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s));
+  GP_CHECK(g, cudaMemsetAsync(g->row_offset, 0, ((uint64_t)g->nr + 1) * 8, s));
+  GP_CHECK(g, cudaMallocAsync((void **)&g->deg, (uint64_t)g->nr * 4 + 4, s));
   if (E > g->tmax[g->h] && !cap_override) {
     g->err = "initial graph exceeds the root bound";
     return GPMA_ERR_INVALID_ARG;
@@ -715,9 +716,9 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
     // (the dense list ek is sorted & unique; place directly)
     GP_LAUNCH(g, k_unique_last, grid_for(m), TB, 0, s, ek, m, keep);  // all ones (unique)
     scan_u32(g, keep, pos, m, s);
-    GP_LAUNCH(g, k_place_edges, grid_for(m), TB, 0, s, ek, ev, pos, keep, m, wk, wv);
+    GP_LAUNCH(g, k_place_edges, grid_for(m), TB, 0, s, ek, ev, pos, keep, m, wk, wv, g->rb);
   }
-  GP_LAUNCH(g, k_place_guards, grid_for(g->V), TB, 0, s, nullptr, g->V, ek, m, wk, wv);
+  GP_LAUNCH(g, k_place_guards, grid_for(g->nr), TB, 0, s, g->rb, g->nr, ek, m, wk, wv);
   GP_CHECK(g, cudaGetLastError());
   return build_from_sorted(g, wk, wv, E, s);
 }
@@ -772,7 +773,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     N = g->ctrl_h->sum;
     uint64_t nl_new = new_cap / g->L;
     GP_LAUNCH(g, k_layout_even, grid_for(new_cap), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
-              g->row_offset, g->L, nl_new);
+              g->row_offset, g->L, nl_new, g->rb);
   }
   GP_LAUNCH(g, k_lvl_keep, gp, TB, 0, s, a);
   scan_u32(g, a.keep, a.kpos, p, s);
@@ -852,6 +853,7 @@ static Lvl make_lvl(gpma *g, int cur, uint64_t p, uint32_t lvl, int op) {
   a.tmax = lvl < g->tmax.size() ? g->tmax[lvl] : 0;
   a.op = op;
   a.force = 0;
+  a.rb = g->rb;
   return a;
 }
 
@@ -940,7 +942,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   if ((st = zero_ctrl(g, s))) return st;
   const uint64_t nl = g->cap / g->L;
   GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt,
-            g->head, (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg);
+            g->head, (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb);
   scan_u32(g, keep, pos, n, s);
   GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, pos + n, 4, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->nunique, &g->ctrl_d->nunique, 8, cudaMemcpyDeviceToHost, s));

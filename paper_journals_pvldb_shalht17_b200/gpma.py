@@ -34,7 +34,7 @@ class gpma_config(C.Structure):
     _fields_ = [("struct_size", C.c_uint32), ("leaf_slots", C.c_uint32), ("initial_capacity", C.c_uint64),
                 ("rho_leaf_bp", C.c_uint16), ("rho_root_bp", C.c_uint16), ("tau_leaf_bp", C.c_uint16),
                 ("tau_root_bp", C.c_uint16), ("init_density_bp", C.c_uint16), ("reserved0", C.c_uint16),
-                ("delete_mode", C.c_uint32)]
+                ("delete_mode", C.c_uint32), ("row_begin", C.c_uint32), ("row_end", C.c_uint32)]
 
 
 class gpma_stats_t(C.Structure):
@@ -73,6 +73,12 @@ def lib() -> C.CDLL:
             "gpma_debug_set_trace": (st, [P, i32]),
             "gpma_debug_trace": (st, [P, P, u64, P]),
             "gpma_kernel_launches": (u64, [P]),
+            "gpma_route": (st, [P, P, P, u64, u32, P, P, P, P]),
+            "gpma_bfs_init": (st, [P, u32, P, P]),
+            "gpma_bfs_level": (st, [P, P, i32, P, P]),
+            "gpma_cc_round": (st, [P, P, i32, P, P]),
+            "gpma_pr_push": (st, [P, P, i32, P, P]),
+            "gpma_pr_update": (st, [P, P, P, C.c_double, P, P]),
             "gpma_debug_profile": (st, [P, C.c_char_p]),
             "gpma_debug_profile_read": (st, [P, C.c_char_p, C.c_size_t]),
             "gpma_status_string": (C.c_char_p, [st]),
@@ -88,7 +94,8 @@ def lib() -> C.CDLL:
 EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destroy", "gpma_update_batch",
            "gpma_bfs", "gpma_cc", "gpma_pagerank", "gpma_pagerank_f32", "gpma_export_csr", "gpma_stats",
            "gpma_debug_dump", "gpma_debug_set_trace", "gpma_debug_trace", "gpma_kernel_launches",
-           "gpma_debug_profile", "gpma_debug_profile_read",
+           "gpma_debug_profile", "gpma_debug_profile_read", "gpma_route", "gpma_bfs_init", "gpma_bfs_level",
+           "gpma_cc_round", "gpma_pr_push", "gpma_pr_update",
            "gpma_status_string", "gpma_last_error"]
 
 
@@ -136,9 +143,11 @@ class Gpma:
     @classmethod
     def gpma_create(cls, num_vertices: int, init_keys=None, init_vals=None, *, leaf_slots: int = 0,
                     initial_capacity: int = 0, delete_mode: int = DELETE_LAZY, thresholds_bp=None,
-                    init_density_bp: int = 6000, stream=None) -> "Gpma":
+                    init_density_bp: int = 6000, rows=None, stream=None) -> "Gpma":
         cfg = gpma_config()
         lib().gpma_config_default(C.byref(cfg))
+        if rows is not None:
+            cfg.row_begin, cfg.row_end = rows
         cfg.leaf_slots = leaf_slots
         cfg.initial_capacity = initial_capacity
         cfg.delete_mode = delete_mode
@@ -251,6 +260,37 @@ class Gpma:
             name, n, ms = line.split("\t")
             out[name] = (int(n), float(ms))
         return out
+
+    # -- sharded-store primitives (device tensors) ---------------------------
+    def gpma_route(self, keys, vals, nranks: int, out_keys, out_vals, stream=None):
+        counts = (C.c_uint64 * nranks)()
+        self._check(lib().gpma_route(self._h, _ptr(keys), _ptr(vals), _numel(keys), nranks, _ptr(out_keys),
+                                     _ptr(out_vals), counts, _stream(stream)), "gpma_route")
+        return [int(c) for c in counts]
+
+    def gpma_bfs_init(self, root: int, levels, stream=None):
+        self._check(lib().gpma_bfs_init(self._h, root, _ptr(levels), _stream(stream)), "gpma_bfs_init")
+
+    def gpma_bfs_level(self, levels, depth: int, stream=None) -> int:
+        f = C.c_uint32(0)
+        self._check(lib().gpma_bfs_level(self._h, _ptr(levels), depth, C.byref(f), _stream(stream)),
+                    "gpma_bfs_level")
+        return f.value
+
+    def gpma_cc_round(self, labels, init: bool, stream=None) -> int:
+        c = C.c_uint64(0)
+        self._check(lib().gpma_cc_round(self._h, _ptr(labels), int(init), C.byref(c), _stream(stream)),
+                    "gpma_cc_round")
+        return c.value
+
+    def gpma_pr_push(self, x, init: bool, y, stream=None):
+        self._check(lib().gpma_pr_push(self._h, _ptr(x), int(init), _ptr(y), _stream(stream)), "gpma_pr_push")
+
+    def gpma_pr_update(self, x, y, damping: float = 0.85, stream=None) -> float:
+        e = C.c_double(0.0)
+        self._check(lib().gpma_pr_update(self._h, _ptr(x), _ptr(y), damping, C.byref(e), _stream(stream)),
+                    "gpma_pr_update")
+        return e.value
 
     def gpma_kernel_launches(self) -> int:
         return int(lib().gpma_kernel_launches(self._h))

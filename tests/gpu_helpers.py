@@ -10,13 +10,13 @@ KEY_NONE = np.uint64(0xFFFFFFFFFFFFFFFF)
 DEV = "cuda:0"
 
 
-def gpu_dump(g):
+def gpu_dump(g, nrows=None):
     st = g.gpma_stats()
     cap, L = st["capacity"], st["leaf_slots"]
     nl = cap // L
     k = torch.empty(cap, dtype=torch.int64, device=DEV)
     v = torch.empty(cap, dtype=torch.int32, device=DEV)
-    ro = torch.empty(g.V + 1, dtype=torch.int64, device=DEV)
+    ro = torch.empty((g.V if nrows is None else nrows) + 1, dtype=torch.int64, device=DEV)
     cnt = torch.empty(nl, dtype=torch.int32, device=DEV)
     hd = torch.empty(nl, dtype=torch.int64, device=DEV)
     g.gpma_debug_dump(k, v, ro, cnt, hd)
@@ -43,7 +43,7 @@ def expected_leaf_live(keys, vals, L):
 
 
 def assert_same_layout(g, o: O.Oracle, guards=True, what=""):
-    gk, gv, gro, gcnt, ghd, st = gpu_dump(g)
+    gk, gv, gro, gcnt, ghd, st = gpu_dump(g, o.nr)
     ok, ov = o.dump()
     assert gk.size == ok.size, f"{what}: capacity {gk.size} != oracle {ok.size}"
     if not np.array_equal(gk, ok):

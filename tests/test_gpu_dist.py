@@ -1,0 +1,93 @@
+"""Sharded (multi-GPU) path on the GPU: CUDA shards + DistGpma orchestration.
+
+Two processes share one B200 through a gloo group (NCCL refuses two ranks on one device);
+every shard's layout must equal an oracle shard fed the same owned batches (bit-exact), and
+the distributed BFS / CC / PageRank must equal the single-store oracle.  A world-size-1 run
+covers the P = 1 path of the same code.
+"""
+import os
+import socket
+
+import numpy as np
+import pytest
+import torch
+
+import oracle as O
+from gpma_gen import bfs_root, config_stream
+
+pytestmark = pytest.mark.gpu
+
+
+def _free_port():
+    with socket.socket() as s:
+        s.bind(("127.0.0.1", 0))
+        return s.getsockname()[1]
+
+
+def _owned(keys, vals, V, P, r):
+    src = keys >> 32
+    m = (src // ((V + P - 1) // P)) == r
+    return keys[m], (None if vals is None else vals[m])
+
+
+def _run(rank, world, port, mode, seed, fails):
+    import torch.distributed as dist
+    from paper_journals_pvldb_shalht17_b200.dist import CudaShard, DistGpma, batch_slice, row_range
+    from tests.gpu_helpers import DEV, assert_same_layout
+    try:
+        if world > 1:
+            os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+            dist.init_process_group("gloo", rank=rank, world_size=world)
+        torch.cuda.set_device(0)
+        sw = config_stream(0, seed=seed)
+        V, W, B = 1024, sw.window, sw.batch
+        k0, v0 = sw.initial()
+        rows = row_range(V, world, rank)
+        lo, hi = batch_slice(W, world, rank)
+        shard = CudaShard(V, rows, DEV, delete_mode=mode)
+        dg = DistGpma(V, k0[lo:hi].contiguous().to(DEV), v0[lo:hi].contiguous().to(DEV), shard)
+        ok0, ov0 = _owned(k0, v0, V, world, rank)
+        osh = O.Oracle(V, ok0, ov0, rows=rows, delete_mode=mode)
+        ref = O.Oracle(V, k0, v0, delete_mode=mode)
+        assert_same_layout(shard.g, osh, what=f"rank {rank} create")
+        x = None
+        for s in range(3):
+            dk, ik, iv = sw.slide(s)
+            a, b = batch_slice(B, world, rank)
+            dg.delete(dk[a:b].contiguous().to(DEV))
+            dg.insert(ik[a:b].contiguous().to(DEV), iv[a:b].contiguous().to(DEV))
+            osh.delete(_owned(dk, None, V, world, rank)[0])
+            osh.insert(*_owned(ik, iv, V, world, rank))
+            ref.delete(dk)
+            ref.insert(ik, iv)
+            assert_same_layout(shard.g, osh, what=f"rank {rank} slide {s}")
+            root = bfs_root(sw, seed, s)
+            assert dg.bfs(root).cpu().numpy().tolist() == ref.bfs(root).tolist(), "BFS"
+            assert dg.cc().cpu().numpy().view(np.uint32).tolist() == ref.cc().tolist(), "CC"
+            xt = None if x is None else torch.from_numpy(x.copy()).to(DEV)
+            xg, it = dg.pagerank(xt, warm=x is not None, tol=0.0, max_iter=6)
+            xo, _ = ref.pagerank(x=x, tol=0.0, max_iter=6)
+            assert it == 6 and np.abs(xg.cpu().numpy() - xo).max() <= 1e-6, "PR"
+            x = xo
+        if world > 1:
+            dist.destroy_process_group()
+    except Exception as e:
+        import traceback
+        fails.put(f"rank {rank}: {e!r}\n{traceback.format_exc()}")
+        raise
+
+
+@pytest.mark.parametrize("mode,seed", [(0, 5), (1, 6)])
+def test_two_shards_one_gpu(mode, seed):
+    import torch.multiprocessing as mp
+    ctx = mp.get_context("spawn")
+    fails = ctx.Queue()
+    mp.spawn(_run, args=(2, _free_port(), mode, seed, fails), nprocs=2, join=True)
+    assert fails.empty()
+
+
+def test_world_size_one_path():
+    import queue
+    q = queue.Queue()
+    _run(0, 1, 0, 0, 9, q)
+    assert q.empty()
