@@ -12,5 +12,5 @@ masking).  See DESIGN.md "Input recipe".
 from .streams import (  # noqa: F401
     KEY_NONE, VAL_TOMB, DST_GUARD,
     splitmix64, draw, rmat_edges, uniform_edges, edge_values, make_stream,
-    SlidingWindow, CONFIGS, config_stream, bfs_root, fig3_layout, fig5_edges,
+    SlidingWindow, CONFIGS, config_stream, weak_scaled, bfs_root, fig3_layout, fig5_edges,
 )

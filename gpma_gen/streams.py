@@ -115,33 +115,50 @@ def edge_values(keys: torch.Tensor, seed: int) -> torch.Tensor:
 
 
 def make_stream(kind: str, V: int, E: int, seed: int, scale: int | None = None,
-                device="cpu") -> torch.Tensor:
+                device="cpu", sub_chunk: int = 1 << 27) -> torch.Tensor:
     """E unique edge keys (int64) in random-timestamp order.
 
-    Draws candidates in chunks of max(E, 4096) until the set of unique, loop-free,
-    in-range edges holds at least E keys; then orders that set by
-    ts = draw(seed_ts, key) (signed int64 order, ties by key) and keeps the first E.
+    Draws candidates in rounds of max(E, 4096) until the set of unique, loop-free, in-range
+    edges holds at least E keys; then orders that set by ts = draw(seed_ts, key) (signed
+    int64 order, ties by key) and keeps the first E.  A round is generated in sub-chunks of
+    `sub_chunk` candidates to bound memory (this does not change the stream).
     """
     new_id = _scramble(V, seed, device)
     chunk = max(E, 4096)
     keys = torch.empty(0, dtype=torch.int64, device=device)
     ctr = 0
     while keys.numel() < E:
-        if kind == "rmat":
-            s, d = rmat_edges(scale, ctr, chunk, seed, device=device)
-        elif kind == "uniform":
-            s, d = uniform_edges(V, ctr, chunk, seed, device=device)
-        else:
-            raise ValueError(kind)
+        parts = [keys]
+        for c0 in range(ctr, ctr + chunk, sub_chunk):
+            cn = min(sub_chunk, ctr + chunk - c0)
+            if kind == "rmat":
+                s, d = rmat_edges(scale, c0, cn, seed, device=device)
+            elif kind == "uniform":
+                s, d = uniform_edges(V, c0, cn, seed, device=device)
+            else:
+                raise ValueError(kind)
+            ok = (s != d) & (s < V) & (d < V)
+            s, d = new_id[s[ok]], new_id[d[ok]]
+            parts.append(torch.unique((s << 32) | d))
+            del s, d, ok
         ctr += chunk
-        ok = (s != d) & (s < V) & (d < V)
-        s, d = new_id[s[ok]], new_id[d[ok]]
-        keys = torch.unique(torch.cat([keys, (s << 32) | d]))
+        keys = torch.unique(torch.cat(parts))
+        del parts
         if ctr > 64 * chunk:
             raise RuntimeError("stream generator: too few unique edges")
     ts = draw(_tag(seed, 0x5453), keys)
     order = torch.argsort(ts, stable=True)       # keys are sorted -> ties broken by key
     return keys[order[:E]].contiguous()
+
+
+def weak_scaled(cfg_index: int, P: int) -> "StreamConfig":
+    """Per-GPU work fixed as P grows (PAPER.md P:1700-1703 style): the RMAT scale grows by
+    log2(P); V, E, window and the global batch all scale by P."""
+    c = CONFIGS[cfg_index]
+    lp = int(math.log2(P))
+    assert 1 << lp == P, "P must be a power of two"
+    return StreamConfig(f"{c.name}-x{P}", c.kind, c.V * P, c.E * P, c.window * P, c.batch * P, c.seed,
+                        scale=None if c.scale is None else c.scale + lp, delete_mode=c.delete_mode)
 
 
 @dataclass
