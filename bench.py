@@ -112,7 +112,7 @@ class Clocks:
 # ------------------------------------------------------------------ algorithmic bytes
 def algo_bytes(kernel: str, cap: int, V: int, L: int, nnz: int, dtype_bytes: int = 8) -> int | None:
     """Algorithmic bytes of ONE launch of the kernel."""
-    if kernel == "k_pr_push":      # read key+val of every slot, contrib once per vertex, y RMW once
+    if kernel in ("k_pr_push", "k_pr_push_win"):  # key+val of every slot, contrib once per vertex, y RMW once
         return 12 * cap + dtype_bytes * V + 2 * dtype_bytes * V
     if kernel == "k_cc_hook":      # read key+val of every slot, parent array read+write once
         return 12 * cap + 8 * V
@@ -203,7 +203,7 @@ def run_gpma(args, rank, world, lrank):
         cap, L = st["capacity"], st["leaf_slots"]
         nnz = st["live_edges"]
         cand = {k: v for k, v in prof_all.items() if algo_bytes(k, cap, V, L, nnz) is not None}
-        dom = max(cand, key=lambda k: cand[k][1]) if cand else "k_pr_push"
+        dom = max(cand, key=lambda k: cand[k][1]) if cand else "k_pr_push_win"
         evs.clear()
         pr_iters.clear()
         g.gpma_debug_profile(dom)
@@ -385,7 +385,7 @@ def run_gpma_dist(args, rank, world, lrank):
             step(i)
             i += 1
         pr_iters.clear()
-        shard.g.gpma_debug_profile("k_pr_push")
+        shard.g.gpma_debug_profile("k_pr_push_win")
         launches0 = shard.g.gpma_kernel_launches()
         dist.barrier()
         torch.cuda.synchronize()
@@ -401,7 +401,7 @@ def run_gpma_dist(args, rank, world, lrank):
         clocks = clk.stop() if clk else None
         ms = e0.elapsed_time(e1)
         launches = shard.g.gpma_kernel_launches() - launches0
-        prof = shard.g.gpma_debug_profile_read().get("k_pr_push", (0, 0.0))
+        prof = shard.g.gpma_debug_profile_read().get("k_pr_push_win", (0, 0.0))
         shard.g.gpma_debug_profile(None)
         e2e = None
         if not args.no_e2e:
@@ -448,7 +448,7 @@ def run_gpma_dist(args, rank, world, lrank):
                    "shard_capacity_rank0": cap,
                    "l2": "no flush: per-GPU store 3.2 GB > 126 MB L2; fresh batch every step"},
         "pr_iters": pr_iters,
-        "roofline": {"bound": "hbm", "kernel": "k_pr_push", "achieved": ach, "peak": hbm, "unit": "GB/s",
+        "roofline": {"bound": "hbm", "kernel": "k_pr_push_win", "achieved": ach, "peak": hbm, "unit": "GB/s",
                      "frac": ach / hbm if ach else None, "traffic": None, "algorithmic_bytes_per_launch": ab,
                      "avg_launch_ms": avg, "launches": n_l, "peak_kind": peak_kind, "rank": 0},
         "e2e": e2e, "gpu_launches": launches, "clocks": clocks, "setup_s": {"generate": gen_s},

@@ -567,6 +567,59 @@ __global__ void __launch_bounds__(TA) k_pr_push(const uint64_t *__restrict__ key
   }
 }
 
+// Row-window push: warp w sweeps the contiguous slot chunk [beg, end) (leaf aligned).  Keys
+// are sorted, so the sources met along the chunk never decrease: lane j keeps contrib[ub + j]
+// of a 32-row window in a register and every slot fetches its source's contribution with a
+// shuffle -- the sweep is a pure key stream plus fire-and-forget REDs, with no dependent
+// global load per slot.  The window moves forward (coalesced 256-B refill) when a source
+// leaves it.
+template <typename A>
+__global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__ key,
+                                                    const uint32_t *__restrict__ tmask,
+                                                    const uint64_t *__restrict__ head, uint32_t L, uint64_t cap,
+                                                    const A *__restrict__ contrib, A *y, uint32_t rb,
+                                                    uint32_t nr) {
+  constexpr int U = 4;                                   // 32-slot groups in flight per warp
+  const int lane = threadIdx.x & 31;
+  const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  const uint64_t w = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32;
+  const uint64_t chunk = (((cap + nwarps - 1) / nwarps) + 32 * U - 1) / (32 * U) * (32 * U);
+  const uint64_t beg = w * chunk, end = min(beg + chunk, cap);
+  if (beg >= end) return;
+  const uint64_t h0 = head[beg / L];
+  if (h0 == KEY_NONE) return;                            // no key at or after this chunk
+  uint32_t ub = (uint32_t)(h0 >> 32) - rb;               // lower bound of the chunk's rows
+  A win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
+  for (uint64_t base = beg; base < end; base += 32 * U) {
+    uint64_t k[U];
+    uint32_t tb[U];
+#pragma unroll
+    for (int j = 0; j < U; ++j) {                       // all loads of the group first
+      const uint64_t s = base + j * 32 + lane;
+      k[j] = s < end ? __ldcs(key + s) : KEY_NONE;
+      tb[j] = s < end ? (__ldg(tmask + s / L) >> (uint32_t)(s % L)) & 1u : 1u;
+    }
+#pragma unroll
+    for (int j = 0; j < U; ++j) {
+      const bool e = live_key(k[j]) && !tb[j];
+      const uint32_t u = (uint32_t)(k[j] >> 32) - rb;
+      uint32_t pending = __ballot_sync(0xffffffffu, e);
+      while (pending) {
+        const bool mine = (pending >> lane) & 1u;
+        const uint32_t off = mine ? u - ub : 0u;
+        const bool in = mine && off < 32u;
+        const A c = __shfl_sync(0xffffffffu, win, off & 31u);
+        if (in) atomicAdd(&y[(uint32_t)k[j]], c);
+        pending &= ~__ballot_sync(0xffffffffu, in);
+        if (pending) {                                   // slide the window to the next source
+          ub = __reduce_min_sync(0xffffffffu, ((pending >> lane) & 1u) ? u : 0xFFFFFFFFu);
+          win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
+        }
+      }
+    }
+  }
+}
+
 // x' = (1-d)/V + d (y + D/V); err += |x'-x|; next contrib / dangling; y := 0
 template <typename T>
 __global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ y,
@@ -608,8 +661,8 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
   int it = 0, cur = 0;
   while (it < max_iter) {
-    GP_LAUNCH(g, k_pr_push<A>, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, contrib, y,
-              0u);
+    GP_LAUNCH(g, k_pr_push_win<A>, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L, g->cap,
+              contrib, y, 0u, g->nr);
     GP_CHECK(g, cudaMemsetAsync(acc + 2, 0, sizeof(double), s));
     GP_CHECK(g, cudaMemsetAsync(acc + (cur ^ 1), 0, sizeof(double), s));
     GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
@@ -673,8 +726,8 @@ gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
   unsigned long long *yy = (unsigned long long *)y;
   if (init) GP_LAUNCH(g, k_prd_init, grid_for(g->V), TA, 0, s, x, g->V);
   GP_LAUNCH(g, k_prd_contrib, grid_for(g->nr), TA, 0, s, x, g->deg, g->rb, g->nr, contrib, yy, g->V);
-  GP_LAUNCH(g, k_pr_push<unsigned long long>, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap,
-            contrib, yy, g->rb);
+  GP_LAUNCH(g, k_pr_push_win<unsigned long long>, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head,
+            g->L, g->cap, contrib, yy, g->rb, g->nr);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
