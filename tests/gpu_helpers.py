@@ -28,13 +28,8 @@ def gpu_dump(g, nrows=None):
 def expected_heads(keys, L):
     """R9 locate index: head[l] = first key of the first non-empty leaf >= l (KEY_NONE if none)."""
     first = keys.reshape(-1, L)[:, 0]
-    out = np.empty_like(first)
-    nxt = KEY_NONE
-    for l in range(first.size - 1, -1, -1):
-        if first[l] != KEY_NONE:
-            nxt = first[l]
-        out[l] = nxt
-    return out
+    # first keys of non-empty leaves increase and KEY_NONE is the maximum: a suffix minimum
+    return np.minimum.accumulate(first[::-1])[::-1]
 
 
 def expected_leaf_live(keys, vals, L):
