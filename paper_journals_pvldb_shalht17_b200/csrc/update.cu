@@ -109,6 +109,165 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
   if ((threadIdx.x & 31) == 0 && u) atomicAdd((unsigned long long *)&c->nunique, (unsigned long long)u);
 }
 
+// Lazy deletion (R12) needs no order: every key of the batch is located and
+// its live slot marked in place.  Duplicates race on the same slot; the CAS on the value
+// lets exactly one of them account the deletion (live count, tombstone bit, out-degree).
+__global__ void k_lazy_delete(const uint64_t *__restrict__ keys, uint64_t n, const uint64_t *__restrict__ key,
+                              uint32_t *val, uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
+                              uint32_t nleaves, uint32_t L, uint32_t *__restrict__ tmask,
+                              uint32_t *__restrict__ deg, uint32_t rb) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    const uint64_t k = keys[i];
+    const uint32_t t = locate_leaf(head, nleaves, k);
+    const uint64_t base = (uint64_t)t * L;
+    for (uint32_t p = 0; p < L; ++p) {
+      const uint64_t x = key[base + p];
+      if (x == k) {
+        uint32_t old = val[base + p];
+        while (old != VAL_TOMB) {
+          const uint32_t seen = atomicCAS(&val[base + p], old, VAL_TOMB);
+          if (seen == old) {
+            atomicSub(&cnt[t], 1u);
+            atomicOr(&tmask[t], 1u << p);
+            atomicSub(&deg[(uint32_t)(k >> 32) - rb], 1u);
+            break;
+          }
+          old = seen;
+        }
+        break;
+      }
+      if (x == KEY_NONE || x > k) break;
+    }
+  }
+}
+
+// Fused level 0 of the level loop (Alg. 4 l.7-15 at the leaves, where nearly every update
+// is absorbed): one warp per group of pending updates that share a target leaf.  The warp
+// loads the leaf (lane l = slot l), counts its live entries with a ballot, tests the leaf
+// bound max_0 (insert) / min_0 (strict delete), and on success merges in registers -- the rank
+// of a live entry is its live rank plus the updates below it, the rank of an update its
+// index plus the live entries below it -- and writes the left-packed leaf back (a one-leaf
+// window has a single piece in the R7 split).  Rejected groups stay pending for level 1.
+__global__ void __launch_bounds__(256) k_level0(const uint64_t *__restrict__ pk, const uint32_t *__restrict__ pv,
+                                                const uint32_t *__restrict__ pt, uint64_t p, uint64_t *key,
+                                                uint32_t *val, uint32_t *__restrict__ cnt,
+                                                uint32_t *__restrict__ tmask, uint64_t *__restrict__ head,
+                                                uint64_t *__restrict__ row_offset, uint32_t rb, uint32_t L,
+                                                uint32_t bound, int op, uint32_t *__restrict__ keep,
+                                                uint2 *__restrict__ dirty, Ctrl *c) {
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  uint32_t accepted = 0;
+  for (uint64_t base = ((blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32) * 32; base < p;
+       base += nwarps * 32) {
+    const uint64_t jl = base + lane;
+    const bool first = jl < p && (jl == 0 || pt[jl] != pt[jl - 1]);
+    uint32_t starts = __ballot_sync(0xffffffffu, first);
+    while (starts) {
+      const int sl = __ffs(starts) - 1;
+      starts &= starts - 1;
+      const uint64_t j0 = base + sl;
+      const uint32_t t = pt[j0];
+      // group end: next start in this window, else scan forward
+      uint64_t j1;
+      if (starts) {
+        j1 = base + (__ffs(starts) - 1);
+      } else {
+        j1 = base + 32;
+        while (true) {                                 // warp-cooperative forward scan
+          const uint64_t jj = j1 + lane;
+          const bool other = jj >= p || pt[jj] != t;
+          const uint32_t b = __ballot_sync(0xffffffffu, other);
+          if (b) { j1 += __ffs(b) - 1; break; }
+          j1 += 32;
+        }
+        if (j1 > p) j1 = p;
+      }
+      const uint32_t u = (uint32_t)(j1 - j0);
+      const uint64_t lb = (uint64_t)t * L;
+      uint64_t ks = KEY_NONE;
+      uint32_t vs = 0;
+      if (lane < (int)L) {
+        ks = key[lb + lane];
+        vs = val[lb + lane];
+      }
+      const bool live = lane < (int)L && ks != KEY_NONE && vs != VAL_TOMB;
+      const uint32_t lb_live = __ballot_sync(0xffffffffu, live);
+      const uint32_t n = __popc(lb_live);
+      bool ok;
+      if (op == GPMA_INSERT) ok = u <= bound && n + u <= bound;
+      else ok = u <= n && n - u >= bound;
+      if (!ok) {
+        for (uint64_t j = j0 + lane; j < j1; j += 32) keep[j] = 1u;
+        continue;
+      }
+      uint64_t uk = KEY_NONE;
+      uint32_t uv = 0;
+      if (lane < (int)u) {
+        uk = pk[j0 + lane];
+        uv = pv[j0 + lane];
+      }
+      // merged ranks
+      uint32_t below_u = 0, below_l = 0;
+      for (uint32_t i = 0; i < u; ++i) below_u += __shfl_sync(0xffffffffu, uk, i) < ks;
+      for (uint32_t i = 0; i < L; ++i) {
+        const uint64_t ki = __shfl_sync(0xffffffffu, ks, i);
+        below_l += ((lb_live >> i) & 1u) && ki < uk;
+      }
+      bool drop = false;                               // (every lane shuffles: full mask)
+      if (op != GPMA_INSERT)
+        for (uint32_t i = 0; i < u; ++i) {
+          const uint64_t ki = __shfl_sync(0xffffffffu, uk, i);   // not short-circuited
+          drop |= live && ki == ks;
+        }
+      const uint32_t N = op == GPMA_INSERT ? n + u : n - u;
+      const uint32_t live_rank = __popc(lb_live & lt);
+      __syncwarp();
+      // new first key of the leaf (held by the lane whose entry lands at position 0)
+      // (a lane may hold both a live entry and an update: pick the one that lands at 0)
+      const bool l0 = live && !drop && (op == GPMA_INSERT ? live_rank + below_u : live_rank - below_u) == 0;
+      const bool u0 = op == GPMA_INSERT && lane < (int)u && lane + below_l == 0;
+      const uint32_t b0 = __ballot_sync(0xffffffffu, l0 || u0);
+      const uint64_t h_new = N ? __shfl_sync(0xffffffffu, l0 ? ks : uk, b0 ? __ffs(b0) - 1 : 0) : KEY_NONE;
+      const uint64_t h_old = __shfl_sync(0xffffffffu, ks, 0);   // first occupied key before
+      // write entries at their merged position, then clear the tail
+      if (live && !drop) {
+        const uint32_t pos = op == GPMA_INSERT ? live_rank + below_u : live_rank - below_u;
+        key[lb + pos] = ks;
+        val[lb + pos] = vs;
+        if (is_guard_key(ks)) row_offset[(ks >> 32) - rb + 1] = lb + pos;
+      }
+      if (op == GPMA_INSERT && lane < (int)u) {
+        const uint32_t pos = lane + below_l;
+        key[lb + pos] = uk;
+        val[lb + pos] = uv;
+      }
+      __syncwarp();
+      if (lane < (int)L && lane >= (int)N) {
+        key[lb + lane] = KEY_NONE;
+        val[lb + lane] = 0;
+      }
+      for (uint64_t j = j0 + lane; j < j1; j += 32) keep[j] = 0u;
+      if (lane == 0) {
+        cnt[t] = N;
+        tmask[t] = 0u;
+        if (h_new != h_old) {
+          head[t] = h_new;
+          // empty leaves to the left carry this head (R9): leave them to the final fix-up
+          if (!N || (t > 0 && key[lb - L] == KEY_NONE)) {
+            const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
+            dirty[d] = make_uint2(t, 1u);
+          }
+        }
+        ++accepted;
+      }
+    }
+  }
+  if (lane == 0 && accepted) atomicAdd((unsigned long long *)&c->windows_rewritten, (unsigned long long)accepted);
+}
+
 __global__ void k_compact_pending(const uint32_t *__restrict__ keep, const uint32_t *__restrict__ pos,
                                   uint64_t n, const uint64_t *__restrict__ ik,
                                   const uint32_t *__restrict__ iv, const uint32_t *__restrict__ it,
@@ -929,6 +1088,14 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   GP_CHECK(g, cudaMemcpyAsync(ik, keys, n * 8, cudaMemcpyDefault, s));
   if (op == GPMA_INSERT) GP_CHECK(g, cudaMemcpyAsync(iv, vals, n * 4, cudaMemcpyDefault, s));
   if ((st = validate(g, ik, iv, n, op == GPMA_INSERT, s))) return st;
+  if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
+    const uint64_t nl0 = g->cap / g->L;
+    GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl0,
+              g->L, tmask_of(g), g->deg, g->rb);
+    g->last.last_unique = n;   // not deduplicated: lazy deletes are idempotent
+    GP_CHECK(g, cudaGetLastError());
+    return GPMA_OK;
+  }
   int which;
   uint64_t m;
   if ((st = sort_unique(g, ik, op == GPMA_INSERT ? iv : nullptr, n, &m, false, &which, s))) return st;
@@ -956,6 +1123,37 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
             (uint64_t *)g->b_pk[0].p, (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p);
   uint64_t dirty_base = 0;
   uint32_t lvl = 0;
+  if (!g->trace_on) {
+    // level 0 fused: one warp per leaf group (the generic step below serves levels >= 1,
+    // and level 0 too when the per-level trace is requested)
+    GP_CHECK(g, cudaMemsetAsync(&g->ctrl_d->ndirty, 0, 16, s));   // ndirty + sum
+    GP_CHECK(g, cudaMemsetAsync(&g->ctrl_d->windows_rewritten, 0, 8, s));
+    uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
+    const uint32_t bound = (uint32_t)(op == GPMA_INSERT ? g->tmax[0] : g->tmin[0]);
+    GP_LAUNCH(g, k_level0, grid_for((p + 31) / 32 * 32), 256, 0, s, (const uint64_t *)g->b_pk[0].p,
+              (const uint32_t *)g->b_pv[0].p, (const uint32_t *)g->b_pt[0].p, p, g->key, g->val, g->cnt,
+              tmask_of(g), g->head, g->row_offset, g->rb, g->L, bound, op, keep2, (uint2 *)g->b_dirty.p,
+              g->ctrl_d);
+    scan_u32(g, keep2, kpos, p, s);
+    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, kpos + p, 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->ndirty, &g->ctrl_d->ndirty, 8, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->windows_rewritten, &g->ctrl_d->windows_rewritten, 8,
+                                cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaStreamSynchronize(s));
+    const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
+    dirty_base = g->ctrl_h->ndirty;
+    g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;
+    g->last.last_windows_rewritten += g->ctrl_h->windows_rewritten;
+    if (p_new) {
+      GP_LAUNCH(g, k_compact_pending, grid_for(p), TB, 0, s, keep2, kpos, p, (const uint64_t *)g->b_pk[0].p,
+                (const uint32_t *)g->b_pv[0].p, (const uint32_t *)g->b_pt[0].p, (uint64_t *)g->b_pk[1].p,
+                (uint32_t *)g->b_pv[1].p, (uint32_t *)g->b_pt[1].p);
+      cur = 1;
+      g->last.last_top_level = 1;
+    }
+    p = p_new;
+    lvl = 1;
+  }
   for (; lvl <= g->h && p > 0; ++lvl) {
     Lvl a = make_lvl(g, cur, p, lvl, op);
     LevelOut lo{};
