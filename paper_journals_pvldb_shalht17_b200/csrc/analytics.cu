@@ -756,17 +756,7 @@ gpma_status pagerank_f32(gpma *g, float *x, int warm, float d, float tol, int ma
 }
 
 // ------------------------------------------------------------------ export CSR
-// guards per leaf from the row offsets (R8: row_offset[u+1] = slot of guard u)
-__global__ void k_exp_guards(const uint64_t *__restrict__ row_offset, const uint64_t *__restrict__ key,
-                             uint32_t rb, uint32_t nr, uint32_t L, uint32_t *__restrict__ gl) {
-  for (uint64_t u = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; u < nr;
-       u += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t s = row_offset[u + 1];
-    if (key[s] == (((u + rb) << 32) | COL_GUARD)) atomicAdd(&gl[s / L], 1u);
-  }
-}
-
-// edges per leaf = live entries (cnt) - guards
+// edges per leaf = live entries - guards (both maintained per leaf by every rewrite)
 __global__ void k_exp_counts(const uint32_t *__restrict__ cnt, const uint32_t *__restrict__ gl, uint64_t nl,
                              uint64_t *__restrict__ lc) {
   for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nl;
@@ -774,16 +764,17 @@ __global__ void k_exp_counts(const uint32_t *__restrict__ cnt, const uint32_t *_
     lc[l] = cnt[l] - gl[l];
 }
 
-// Compaction sweep, 4 slots per thread: rank = leaf base + edges before this slot in the
-// leaf (exclusive scan over the L/4 lanes that share the leaf + the thread's own slots).
+// Compaction sweep, 4 slots per thread.  A warp's 128 slots are leaf aligned and their
+// edges land contiguously in the output from lbase[first leaf]: ranks come from a warp scan,
+// the (col, val) pairs are staged in shared memory and stored as full coalesced lines.
 __global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ key,
                                                   const uint32_t *__restrict__ val,
                                                   const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
                                                   const uint64_t *__restrict__ lbase,
                                                   uint64_t *__restrict__ row_ptr, uint32_t *__restrict__ col,
                                                   uint32_t *__restrict__ cval, uint32_t rb) {
-  const int lane = threadIdx.x & 31;
-  const uint32_t lpl = L / 4;                    // lanes per leaf (1..8)
+  __shared__ uint32_t s_col[TA / 32][128], s_val[TA / 32][128];
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   const uint64_t n4 = cap / 4, n4r = (n4 + 31) & ~31ull;
   for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4r;
        t += (uint64_t)gridDim.x * blockDim.x) {
@@ -793,27 +784,38 @@ __global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ k
       load4(key, tmask, L, t * 4, sl);
 #pragma unroll
       for (int j = 0; j < 4; ++j) e |= (edge4(sl, j) ? 1u : 0u) << j;
+    } else {
+      sl.k[0] = sl.k[1] = sl.k[2] = sl.k[3] = KEY_NONE;
     }
-    uint32_t c = __popc(e), incl = c;
-    for (uint32_t o = 1; o < lpl; o <<= 1) {
+    const uint32_t c = __popc(e);
+    uint32_t incl = c;
+    for (int o = 1; o < 32; o <<= 1) {
       uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
-      if ((lane % lpl) >= o) incl += y;
+      if (lane >= o) incl += y;
     }
-    if (t >= n4) continue;
-    uint64_t r = lbase[(t * 4) / L] + incl - c;
+    const uint32_t total = __shfl_sync(0xffffffffu, incl, 31);
+    const uint64_t t0 = t - lane;                               // warp's first slot group
+    const uint64_t wbase = t0 < n4 ? lbase[(t0 * 4) / L] : 0;
     uint4 vv = make_uint4(0, 0, 0, 0);
     if (e) vv = __ldcs(reinterpret_cast<const uint4 *>(val + t * 4));
     const uint32_t vs[4] = {vv.x, vv.y, vv.z, vv.w};
+    uint32_t r = incl - c;
 #pragma unroll
     for (int j = 0; j < 4; ++j) {
       if ((e >> j) & 1u) {
-        col[r] = (uint32_t)sl.k[j];
-        cval[r] = vs[j];
+        s_col[w][r] = (uint32_t)sl.k[j];
+        s_val[w][r] = vs[j];
         ++r;
       } else if (is_guard_key(sl.k[j])) {
-        row_ptr[(sl.k[j] >> 32) - rb + 1] = r;
+        row_ptr[(sl.k[j] >> 32) - rb + 1] = wbase + r;
       }
     }
+    __syncwarp();
+    for (uint32_t i = lane; i < total; i += 32) {
+      col[wbase + i] = s_col[w][i];
+      cval[wbase + i] = s_val[w][i];
+    }
+    __syncwarp();
   }
 }
 
@@ -821,12 +823,8 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
                        uint64_t *nnz_out, cudaStream_t s) {
   const uint64_t nl = g->cap / g->L;
   GP_CHECK(g, ensure(g->b_lpre, (nl + 1) * 8, s));
-  GP_CHECK(g, ensure(g->b_an[0], (nl + 1) * 4, s));
   uint64_t *lc = (uint64_t *)g->b_lpre.p;
-  uint32_t *gl = (uint32_t *)g->b_an[0].p;
-  GP_CHECK(g, cudaMemsetAsync(gl, 0, nl * 4, s));
-  GP_LAUNCH(g, k_exp_guards, grid_for(g->nr), TA, 0, s, g->row_offset, g->key, g->rb, g->nr, g->L, gl);
-  GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gl, nl, lc);
+  GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gcnt_of(g), nl, lc);
   scan_u64(g, lc, lc, nl, s);
   GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, lc + nl, 8, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaStreamSynchronize(s));

@@ -213,7 +213,7 @@ gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t l
     gp::level_bounds(g->L, g->h, g->rho0, g->rhoh, g->tau0, g->tauh, g->tmin, g->tmax);
     uint64_t nl = capacity / leaf_slots;
     if (cudaMallocAsync((void **)&g->key, capacity * 8, s) || cudaMallocAsync((void **)&g->val, capacity * 4, s) ||
-        cudaMallocAsync((void **)&g->cnt, nl * 8, s) || cudaMallocAsync((void **)&g->head, nl * 8, s) ||
+        cudaMallocAsync((void **)&g->cnt, nl * 12, s) || cudaMallocAsync((void **)&g->head, nl * 8, s) ||
         cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s) ||
         cudaMallocAsync((void **)&g->deg, (uint64_t)g->nr * 4 + 4, s)) {
       cudaGetLastError();

@@ -65,8 +65,9 @@ struct gpma {
   // store (HBM-resident)
   uint64_t *key = nullptr;        // [cap]
   uint32_t *val = nullptr;        // [cap]
-  uint32_t *cnt = nullptr;        // [2*cap/L]: live entries (incl. guards) per leaf, then the
-                                  // per-leaf tombstone bit mask (bit p = slot p is a tombstone)
+  uint32_t *cnt = nullptr;        // [3*cap/L]: live entries (incl. guards) per leaf, then the
+                                  // per-leaf tombstone bit mask (bit p = slot p is a tombstone),
+                                  // then the guards per leaf
   uint32_t *deg = nullptr;        // [V] live out-degree per vertex, maintained by every batch
   uint64_t *head = nullptr;       // [cap/L] locate index (R9)
   uint64_t *row_offset = nullptr; // [V+1] (R8)
@@ -162,6 +163,7 @@ gpma_status recompute_heads(gpma *g, cudaStream_t s);
 gpma_status count_slots(gpma *g, uint64_t *live_edges, uint64_t *tombs, cudaStream_t s);
 gpma_status recompute_degrees(gpma *g, cudaStream_t s);   // analytics.cu
 inline uint32_t *tmask_of(gpma *g) { return g->cnt + g->cap / g->L; }
+inline uint32_t *gcnt_of(gpma *g) { return g->cnt + 2 * (g->cap / g->L); }
 
 // analytics (analytics.cu)
 gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s);

@@ -300,6 +300,7 @@ struct Lvl {
   int op;
   int force;           // resize: accept the single root window unconditionally
   uint32_t rb;         // first owned row (row offsets are local)
+  uint64_t nleaves;    // leaves of the store (offset of the guard counts after the masks)
 };
 
 __global__ void k_lvl_flags(Lvl a) {
@@ -507,6 +508,9 @@ __global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *
     if (p == 0) {
       cnt[leaf0 + l] = (uint32_t)(hi - lo);
       tmask[leaf0 + l] = 0u;                          // tombstones are dropped by a rewrite
+      uint32_t gc = 0;
+      for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(a.wk[a.woff[w] + e]);
+      tmask[a.nleaves + leaf0 + l] = gc;              // guards per leaf (third section)
     }
     if (off == 0) dirty[dirty_base + ai] = make_uint2((uint32_t)leaf0, (uint32_t)Lc);
   }
@@ -549,6 +553,9 @@ __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *_
     if (p == 0) {
       cnt[l] = (uint32_t)(hi - lo);
       tmask[l] = 0u;
+      uint32_t gc = 0;
+      for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(wk[e]);
+      tmask[nleaves + l] = gc;
     }
   }
 }
@@ -672,17 +679,19 @@ __global__ void k_raw_counts(const uint64_t *__restrict__ key, const uint32_t *_
                              uint64_t nleaves, uint32_t rb, uint32_t nr) {
   for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
        l += (uint64_t)gridDim.x * blockDim.x) {
-    uint32_t c = 0, m = 0;
+    uint32_t c = 0, m = 0, gc = 0;
     for (uint32_t p = 0; p < L; ++p) {
       uint64_t s = l * L + p;
       uint64_t k = key[s];
       if (k == KEY_NONE) continue;
+      gc += is_guard_key(k);
       if (val[s] != VAL_TOMB) ++c;
       else m |= 1u << p;
       if (is_guard_key(k) && (uint32_t)(k >> 32) - rb < nr) row_offset[(k >> 32) - rb + 1] = s;
     }
     cnt[l] = c;
     cnt[nleaves + l] = m;
+    cnt[2 * nleaves + l] = gc;
   }
 }
 
@@ -727,7 +736,7 @@ static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v
   *k = nullptr; *v = nullptr; *c = nullptr; *hd = nullptr;
   cudaError_t e1 = cudaMallocAsync((void **)k, cap * 8, s);
   cudaError_t e2 = cudaMallocAsync((void **)v, cap * 4, s);
-  cudaError_t e3 = cudaMallocAsync((void **)c, nl * 8, s);   // live counts + tombstone masks
+  cudaError_t e3 = cudaMallocAsync((void **)c, nl * 12, s);  // live counts, tombstone masks, guards
   cudaError_t e4 = cudaMallocAsync((void **)hd, nl * 8, s);
   if (e1 || e2 || e3 || e4) {
     cudaGetLastError();
@@ -1013,6 +1022,7 @@ static Lvl make_lvl(gpma *g, int cur, uint64_t p, uint32_t lvl, int op) {
   a.op = op;
   a.force = 0;
   a.rb = g->rb;
+  a.nleaves = g->cap / g->L;
   return a;
 }
 
