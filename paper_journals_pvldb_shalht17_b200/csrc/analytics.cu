@@ -23,6 +23,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cstdlib>
 #include <cstring>
 
 #include "gpma_internal.cuh"
@@ -574,13 +575,12 @@ __global__ void __launch_bounds__(TA) k_pr_push(const uint64_t *__restrict__ key
 // shuffle -- the sweep is a pure key stream plus fire-and-forget REDs, with no dependent
 // global load per slot.  The window moves forward (coalesced 256-B refill) when a source
 // leaves it.
-template <typename A>
+template <typename A, int U>
 __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__ key,
                                                     const uint32_t *__restrict__ tmask,
                                                     const uint64_t *__restrict__ head, uint32_t L, uint64_t cap,
                                                     const A *__restrict__ contrib, A *y, uint32_t rb,
-                                                    uint32_t nr) {
-  constexpr int U = 4;                                   // 32-slot groups in flight per warp
+                                                    uint32_t nr, uint32_t dlo, uint32_t dhi) {
   const int lane = threadIdx.x & 31;
   const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
   const uint64_t w = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32;
@@ -591,18 +591,23 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
   if (h0 == KEY_NONE) return;                            // no key at or after this chunk
   uint32_t ub = (uint32_t)(h0 >> 32) - rb;               // lower bound of the chunk's rows
   A win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
-  for (uint64_t base = beg; base < end; base += 32 * U) {
-    uint64_t k[U];
-    uint32_t tb[U];
-#pragma unroll
-    for (int j = 0; j < U; ++j) {                       // all loads of the group first
-      const uint64_t s = base + j * 32 + lane;
-      k[j] = s < end ? __ldcs(key + s) : KEY_NONE;
-      tb[j] = s < end ? (__ldg(tmask + s / L) >> (uint32_t)(s % L)) & 1u : 1u;
-    }
+  uint64_t k[U], kn[U];
+  uint32_t tb[U], tbn[U];
+  auto fetch = [&](uint64_t base, uint64_t *kk, uint32_t *tt) {
 #pragma unroll
     for (int j = 0; j < U; ++j) {
-      const bool e = live_key(k[j]) && !tb[j];
+      const uint64_t s = base + j * 32 + lane;
+      kk[j] = s < end ? __ldcs(key + s) : KEY_NONE;
+      tt[j] = s < end ? (__ldg(tmask + s / L) >> (uint32_t)(s % L)) & 1u : 1u;
+    }
+  };
+  fetch(beg, k, tb);
+  for (uint64_t base = beg; base < end; base += 32 * U) {
+    if (base + 32 * U < end) fetch(base + 32 * U, kn, tbn);      // next group in flight
+#pragma unroll
+    for (int j = 0; j < U; ++j) {
+      const uint32_t dv = (uint32_t)k[j];
+      const bool e = live_key(k[j]) && !tb[j] && dv >= dlo && dv < dhi;   // this pass's targets
       const uint32_t u = (uint32_t)(k[j] >> 32) - rb;
       uint32_t pending = __ballot_sync(0xffffffffu, e);
       while (pending) {
@@ -610,13 +615,18 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
         const uint32_t off = mine ? u - ub : 0u;
         const bool in = mine && off < 32u;
         const A c = __shfl_sync(0xffffffffu, win, off & 31u);
-        if (in) atomicAdd(&y[(uint32_t)k[j]], c);
+        if (in) atomicAdd(&y[dv], c);
         pending &= ~__ballot_sync(0xffffffffu, in);
         if (pending) {                                   // slide the window to the next source
           ub = __reduce_min_sync(0xffffffffu, ((pending >> lane) & 1u) ? u : 0xFFFFFFFFu);
           win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
         }
       }
+    }
+#pragma unroll
+    for (int j = 0; j < U; ++j) {
+      k[j] = kn[j];
+      tb[j] = tbn[j];
     }
   }
 }
@@ -647,6 +657,16 @@ __global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ 
   }
 }
 
+// Destination passes of the push (GPMA_PR_PASSES, default 1).  Random REDs run ~3x faster
+// while their target fits in L2 (tools/micro/red_bench.cu), but each pass re-sweeps the keys;
+// at V = 2^24 one pass measured fastest.
+static uint32_t pr_passes(uint64_t ybytes) {
+  (void)ybytes;
+  uint64_t p = 1;
+  if (const char *e = getenv("GPMA_PR_PASSES")) p = (uint64_t)atoi(e);
+  return (uint32_t)std::max<uint64_t>(1, std::min<uint64_t>(p, 8));
+}
+
 template <typename T>
 static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_iter, int *iters,
                               cudaStream_t s) {
@@ -658,12 +678,15 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   const uint32_t *deg = g->deg;
   A *contrib = (A *)g->b_an[1].p, *y = (A *)g->b_an[2].p;
   double *acc = (double *)g->b_an[3].p;   // [0],[1] dangling ping-pong, [2] error
+  const uint32_t passes = pr_passes(V * sizeof(A));
   GP_CHECK(g, cudaMemsetAsync(acc, 0, 4 * sizeof(double), s));
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
   int it = 0, cur = 0;
   while (it < max_iter) {
-    GP_LAUNCH(g, k_pr_push_win<A>, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L, g->cap,
-              contrib, y, 0u, g->nr);
+    // destination passes: random REDs run ~3x faster while their target fits in L2
+    for (uint32_t q = 0; q < passes; ++q)
+      GP_LAUNCH(g, (k_pr_push_win<A, 4>), MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
+                g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes));
     GP_CHECK(g, cudaMemsetAsync(acc + 2, 0, sizeof(double), s));
     GP_CHECK(g, cudaMemsetAsync(acc + (cur ^ 1), 0, sizeof(double), s));
     GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
@@ -727,8 +750,11 @@ gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
   unsigned long long *yy = (unsigned long long *)y;
   if (init) GP_LAUNCH(g, k_prd_init, grid_for(g->V), TA, 0, s, x, g->V);
   GP_LAUNCH(g, k_prd_contrib, grid_for(g->nr), TA, 0, s, x, g->deg, g->rb, g->nr, contrib, yy, g->V);
-  GP_LAUNCH(g, k_pr_push_win<unsigned long long>, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head,
-            g->L, g->cap, contrib, yy, g->rb, g->nr);
+  const uint32_t passes = pr_passes((uint64_t)g->V * 8);
+  for (uint32_t q = 0; q < passes; ++q)
+    GP_LAUNCH(g, (k_pr_push_win<unsigned long long, 4>), MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g),
+              g->head, g->L, g->cap, contrib, yy, g->rb, g->nr, (uint32_t)((uint64_t)g->V * q / passes),
+              (uint32_t)((uint64_t)g->V * (q + 1) / passes));
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }

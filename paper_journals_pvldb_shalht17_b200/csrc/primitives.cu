@@ -46,6 +46,7 @@ static size_t take_event(gpma *g) {
 }
 
 bool prof_begin(gpma *g, const char *name, cudaStream_t s) {
+  while (*name == '(') ++name;            // GP_LAUNCH((k<T, U>), ...) stringises the parentheses
   if (g->prof_filter != "*") {
     // exact match on the kernel name without template arguments
     const char *lt = strchr(name, '<');
