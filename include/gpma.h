@@ -161,6 +161,25 @@ gpma_status gpma_debug_set_trace(gpma_t *g, int enable);
  * carries the final offset.  Returns the record count in *count; copies at most max. */
 gpma_status gpma_debug_trace(gpma_t *g, uint64_t *out4, uint64_t max, uint64_t *count);
 
+/* ---------------------------------------------------------------- query buffer
+ * Batched ad-hoc queries on the live store (the dynamic query buffer, §3). */
+
+/* Edge lookup: keys u64[n] -> vals u32[n] (0xFFFFFFFF if absent or deleted) and found u8[n]
+ * (either output may be NULL). */
+gpma_status gpma_query_edges(gpma_t *g, const uint64_t *keys, uint64_t n, uint32_t *vals, uint8_t *found,
+                             gpma_stream_t stream);
+/* Neighbourhoods: the live out-edges of verts u32[n] as a CSR -- row_ptr u64[n+1],
+ * col u32[nnz], val u32[nnz] (val may be NULL), rows in query order, columns in key order.
+ * col == NULL: only *nnz_out (size query).  Not available on sharded stores for rows they
+ * do not own (those rows come back empty). */
+gpma_status gpma_query_neighbors(gpma_t *g, const uint32_t *verts, uint64_t n, uint64_t *row_ptr, uint32_t *col,
+                                 uint32_t *val, uint64_t nnz_capacity, uint64_t *nnz_out, gpma_stream_t stream);
+/* Reachability of pairs: reachable u8[n] = 1 iff a directed path src[i] -> dst[i] exists over the
+ * live edges ("check the dynamic reachability between pairs of vertices"); a
+ * multi-source BFS answers 64 pairs per sweep.  Unsharded stores only. */
+gpma_status gpma_query_reachable(gpma_t *g, const uint32_t *src, const uint32_t *dst, uint64_t n,
+                                 uint8_t *reachable, gpma_stream_t stream);
+
 /* ---------------------------------------------------------------- sharded stores
  * Multi-GPU ("evenly partition graphs according to the vertex index and
  * synchronize all devices after each iteration"; R24): one store per rank holds

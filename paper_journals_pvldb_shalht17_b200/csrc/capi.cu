@@ -423,6 +423,70 @@ gpma_status gpma_debug_profile_read(gpma_t *g, char *buf, size_t buflen) {
   return GPMA_OK;
 }
 
+// ---- query buffer
+gpma_status gpma_query_edges(gpma_t *g, const uint64_t *keys, uint64_t n, uint32_t *vals, uint8_t *found,
+                             gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (n && !keys) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  Out ov(g, vals, (size_t)n * 4, s), of(g, found, (size_t)n, s);
+  void *dv, *df;
+  if (cudaError_t e = ov.dev(&dv, false)) return gp::cuda_fail(g, e, "query staging");
+  if (cudaError_t e = of.dev(&df, false)) return gp::cuda_fail(g, e, "query staging");
+  st = gp::query_edges(g, keys, n, (uint32_t *)dv, (uint8_t *)df, s);
+  if (st == GPMA_OK) {
+    cudaError_t e;
+    if ((e = ov.finish()) || (e = of.finish())) return gp::cuda_fail(g, e, "query copy-out");
+  }
+  return end(g, st);
+}
+
+gpma_status gpma_query_neighbors(gpma_t *g, const uint32_t *verts, uint64_t n, uint64_t *row_ptr, uint32_t *col,
+                                 uint32_t *val, uint64_t nnz_capacity, uint64_t *nnz_out, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if ((n && !verts) || (col && !row_ptr)) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  uint64_t nnz = 0;
+  if (!col) {
+    st = gp::query_neighbors(g, verts, n, nullptr, nullptr, nullptr, 0, &nnz, s);
+    if (nnz_out) *nnz_out = nnz;
+    return end(g, st);
+  }
+  Out orp(g, row_ptr, ((size_t)n + 1) * 8, s), oc(g, col, (size_t)nnz_capacity * 4, s),
+      ov(g, val, (size_t)nnz_capacity * 4, s);
+  void *drp, *dc, *dv;
+  if (cudaError_t e = orp.dev(&drp, false)) return gp::cuda_fail(g, e, "query staging");
+  if (cudaError_t e = oc.dev(&dc, false)) return gp::cuda_fail(g, e, "query staging");
+  if (cudaError_t e = ov.dev(&dv, false)) return gp::cuda_fail(g, e, "query staging");
+  st = gp::query_neighbors(g, verts, n, (uint64_t *)drp, (uint32_t *)dc, (uint32_t *)dv, nnz_capacity, &nnz, s);
+  if (nnz_out) *nnz_out = nnz;
+  if (st == GPMA_OK) {
+    oc.bytes = (size_t)nnz * 4;
+    ov.bytes = (size_t)nnz * 4;
+    cudaError_t e;
+    if ((e = orp.finish()) || (e = oc.finish()) || (e = ov.finish())) return gp::cuda_fail(g, e, "query copy-out");
+  }
+  return end(g, st);
+}
+
+gpma_status gpma_query_reachable(gpma_t *g, const uint32_t *src, const uint32_t *dst, uint64_t n, uint8_t *reachable,
+                                 gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (n && (!src || !dst || !reachable)) return GPMA_ERR_INVALID_ARG;
+  if (g->nr != g->V) return GPMA_ERR_INVALID_ARG;
+  cudaStream_t s = (cudaStream_t)stream;
+  Out o(g, reachable, (size_t)n, s);
+  void *d;
+  if (cudaError_t e = o.dev(&d, false)) return gp::cuda_fail(g, e, "query staging");
+  st = gp::query_reachable(g, src, dst, n, (uint8_t *)d, s);
+  if (st == GPMA_OK)
+    if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "query copy-out");
+  return end(g, st);
+}
+
 // ---- sharded-store primitives (device pointers)
 gpma_status gpma_route(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, uint32_t nranks,
                        uint64_t *out_keys, uint32_t *out_vals, uint64_t *counts, gpma_stream_t stream) {

@@ -134,6 +134,12 @@ int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t
 gpma_status radix_partition_owner(gpma *g, const uint64_t *k0, const uint32_t *v0, uint64_t *k1, uint32_t *v1,
                                   uint64_t n, uint32_t div, uint32_t nranks, uint64_t *starts_dev,
                                   cudaStream_t s);
+// query buffer (query.cu)
+gpma_status query_edges(gpma *g, const uint64_t *keys, uint64_t n, uint32_t *vals, uint8_t *found, cudaStream_t s);
+gpma_status query_neighbors(gpma *g, const uint32_t *verts, uint64_t n, uint64_t *row_ptr, uint32_t *col,
+                            uint32_t *val, uint64_t cap_nnz, uint64_t *nnz_out, cudaStream_t s);
+gpma_status query_reachable(gpma *g, const uint32_t *src, const uint32_t *dst, uint64_t n, uint8_t *out,
+                            cudaStream_t s);
 // distributed primitives (dist.cu / analytics.cu)
 gpma_status route(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, uint32_t nranks,
                   uint64_t *out_keys, uint32_t *out_vals, uint64_t *counts_host, cudaStream_t s);

@@ -74,6 +74,9 @@ def lib() -> C.CDLL:
             "gpma_debug_trace": (st, [P, P, u64, P]),
             "gpma_kernel_launches": (u64, [P]),
             "gpma_route": (st, [P, P, P, u64, u32, P, P, P, P]),
+            "gpma_query_edges": (st, [P, P, u64, P, P, P]),
+            "gpma_query_neighbors": (st, [P, P, u64, P, P, P, u64, P, P]),
+            "gpma_query_reachable": (st, [P, P, P, u64, P, P]),
             "gpma_bfs_init": (st, [P, u32, P, P]),
             "gpma_bfs_level": (st, [P, P, i32, P, P]),
             "gpma_cc_round": (st, [P, P, i32, P, P]),
@@ -95,7 +98,8 @@ EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destro
            "gpma_bfs", "gpma_cc", "gpma_pagerank", "gpma_pagerank_f32", "gpma_export_csr", "gpma_stats",
            "gpma_debug_dump", "gpma_debug_set_trace", "gpma_debug_trace", "gpma_kernel_launches",
            "gpma_debug_profile", "gpma_debug_profile_read", "gpma_route", "gpma_bfs_init", "gpma_bfs_level",
-           "gpma_cc_round", "gpma_pr_push", "gpma_pr_update",
+           "gpma_cc_round", "gpma_pr_push", "gpma_pr_update", "gpma_query_edges", "gpma_query_neighbors",
+           "gpma_query_reachable",
            "gpma_status_string", "gpma_last_error"]
 
 
@@ -259,6 +263,24 @@ class Gpma:
         for line in buf.value.decode().splitlines():
             name, n, ms = line.split("\t")
             out[name] = (int(n), float(ms))
+        return out
+
+    # -- query buffer ---------------------------------------------------------
+    def gpma_query_edges(self, keys, vals=None, found=None, stream=None):
+        self._check(lib().gpma_query_edges(self._h, _ptr(keys), _numel(keys), _ptr(vals), _ptr(found),
+                                           _stream(stream)), "gpma_query_edges")
+
+    def gpma_query_neighbors(self, verts, row_ptr=None, col=None, val=None, stream=None) -> int:
+        nnz = C.c_uint64(0)
+        cap = 0 if col is None else _numel(col)
+        self._check(lib().gpma_query_neighbors(self._h, _ptr(verts), _numel(verts), _ptr(row_ptr), _ptr(col),
+                                               _ptr(val), cap, C.byref(nnz), _stream(stream)),
+                    "gpma_query_neighbors")
+        return nnz.value
+
+    def gpma_query_reachable(self, src, dst, out, stream=None):
+        self._check(lib().gpma_query_reachable(self._h, _ptr(src), _ptr(dst), _numel(src), _ptr(out),
+                                               _stream(stream)), "gpma_query_reachable")
         return out
 
     # -- sharded-store primitives (device tensors) ---------------------------
