@@ -1,0 +1,90 @@
+"""Transfer-hiding sliding-window driver (§3 Fig. 2).
+
+"by repeating the aforementioned process, all data transfers are overlapped with concurrent
+device computations".  Slide i's update + analytics run on the compute stream
+through the C ABI (device buffers), while a copy stream moves slide i+1's batches host->device
+and slide i-1's results device->host; events order the two streams.  Pure plumbing: every
+step of the method still runs in libgpma's kernels.
+"""
+from __future__ import annotations
+
+import torch
+
+
+class SlidingWindowPipeline:
+    def __init__(self, g, V: int, max_batch: int, nnz_capacity: int, device, rows: int | None = None,
+                 pr_tol: float = 1e-3):
+        self.g, self.V, self.dev, self.pr_tol = g, V, torch.device(device), pr_tol
+        self.cs = torch.cuda.Stream(self.dev)      # compute
+        self.xs = torch.cuda.Stream(self.dev)      # copies
+        nr = V if rows is None else rows
+        B = max_batch
+        mk = lambda n, dt: torch.empty(n, dtype=dt, device=self.dev)
+        self.d_in = [(mk(B, torch.int64), mk(B, torch.int64), mk(B, torch.int32)) for _ in range(2)]
+        self.n_in = [(0, 0), (0, 0)]
+        self.ev_in = [torch.cuda.Event() for _ in range(2)]
+        # results of the previous slide are read from the second buffer while this one is written
+        self.d_out = [(mk(V, torch.int32), mk(V, torch.int32), mk(nr + 1, torch.int64),
+                       mk(nnz_capacity, torch.int32), mk(nnz_capacity, torch.int32)) for _ in range(2)]
+        self.x = mk(V, torch.float64)
+        self.d_x = [mk(V, torch.float64) for _ in range(2)]
+        self.ev_done = [torch.cuda.Event() for _ in range(2)]
+        self.ev_out = [torch.cuda.Event() for _ in range(2)]
+        pin = lambda t: torch.empty(t.shape, dtype=t.dtype, pin_memory=True)
+        self.h_out = [tuple(pin(t) for t in self.d_out[0]) + (pin(self.x),) for _ in range(2)]
+        self.nnz = [0, 0]
+        self.pr_iters = []
+        self.i = 0
+        with torch.cuda.stream(self.cs):
+            g.gpma_pagerank(self.x, warm_start=False, tol_l1=pr_tol, stream=self.cs)
+
+    def stage(self, slot: int, dk, ik, iv):
+        """Queue the H2D of one slide's batches (pinned host tensors) on the copy stream."""
+        kd, ki, vi = self.d_in[slot]
+        if slot < 2:
+            self.xs.wait_event(self.ev_done[slot])   # the buffer's previous slide is consumed
+        with torch.cuda.stream(self.xs):
+            kd[: dk.numel()].copy_(dk, non_blocking=True)
+            ki[: ik.numel()].copy_(ik, non_blocking=True)
+            vi[: iv.numel()].copy_(iv, non_blocking=True)
+            self.ev_in[slot].record(self.xs)
+        self.n_in[slot] = (dk.numel(), ik.numel())
+
+    def run(self, slot: int, root: int):
+        """Slide on the compute stream, then queue its results' D2H on the copy stream."""
+        g, s = self.g, self.cs
+        kd, ki, vi = self.d_in[slot]
+        nd, ni = self.n_in[slot]
+        lv, lab, rp, col, cv = self.d_out[slot]
+        s.wait_event(self.ev_in[slot])
+        s.wait_event(self.ev_out[slot])          # host copy of this buffer's last results is done
+        with torch.cuda.stream(s):
+            g.gpma_update_batch(kd[:nd], None, 1, stream=s)
+            g.gpma_update_batch(ki[:ni], vi[:ni], 0, stream=s)
+            g.gpma_bfs(root, lv, stream=s)
+            g.gpma_cc(lab, stream=s)
+            self.pr_iters.append(g.gpma_pagerank(self.x, warm_start=True, tol_l1=self.pr_tol, stream=s))
+            self.d_x[slot].copy_(self.x, non_blocking=True)
+            self.nnz[slot] = g.gpma_export_csr(rp, col, cv, stream=s)
+            self.ev_done[slot].record(s)
+        self.xs.wait_event(self.ev_done[slot])
+        h = self.h_out[slot]
+        n = self.nnz[slot]
+        with torch.cuda.stream(self.xs):
+            h[0].copy_(lv, non_blocking=True)
+            h[1].copy_(lab, non_blocking=True)
+            h[2].copy_(rp, non_blocking=True)
+            h[3][:n].copy_(col[:n], non_blocking=True)
+            h[4][:n].copy_(cv[:n], non_blocking=True)
+            h[5].copy_(self.d_x[slot], non_blocking=True)
+            self.ev_out[slot].record(self.xs)
+
+    def results(self, slot: int):
+        """Host results of the slide that last ran in `slot` (waits for their copies)."""
+        self.ev_out[slot].synchronize()
+        lv, lab, rp, col, cv, x = self.h_out[slot]
+        n = self.nnz[slot]
+        return lv, lab, rp, col[:n], cv[:n], x
+
+    def drain(self):
+        torch.cuda.synchronize(self.dev)
