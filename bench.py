@@ -54,6 +54,7 @@ def parse():
     ap.add_argument("--ref-sample-batch", type=int, default=1 << 16)
     ap.add_argument("--profile-all", action="store_true", help="print the per-kernel time table")
     ap.add_argument("--force-dist", action="store_true", help="use the sharded path even at N=1 (testing)")
+    ap.add_argument("--no-sweep", action="store_true", help="skip the configs[1] batch-size sweep")
     return ap.parse_args()
 
 
@@ -329,9 +330,53 @@ def run_gpma(args, rank, world, lrank):
     if args.profile_all:
         out["kernel_table_warm_step"] = {k: {"launches": v[0], "ms": v[1]} for k, v in
                                          sorted(prof_all.items(), key=lambda kv: -kv[1][1])}
+    if not args.no_sweep:
+        del sw, g
+        torch.cuda.empty_cache()
+        out["batch_sweep"] = batch_sweep(dev)
     if world == 1 and not args.no_cpu_baseline:
-        out["cpu_baseline"] = cpu_baseline(sw, cfg, args, 0)
+        out["cpu_baseline"] = cpu_baseline(config_stream(args.config, device=dev), cfg, args, 0)
     print(json.dumps(out))
+
+
+def batch_sweep(dev, batches=(100, 1_000, 10_000, 100_000, 1_000_000)):
+    """Update throughput vs batch size (Fig. 7) on configs[1]
+    (Pokec-shaped, 15M-edge window): per B a fresh store from the initial window, 3 warm-up
+    slides, then slides until >= 2M updates (>= 10 slides); slide = DELETE(B oldest) +
+    INSERT(B next), CUDA-event timed."""
+    from paper_journals_pvldb_shalht17_b200 import Gpma
+    cfg = CONFIGS[1]
+    sw = config_stream(1, device=dev)
+    res = []
+    s = torch.cuda.Stream(dev)
+    avail = sw.keys.numel() - sw.window
+    with torch.cuda.stream(s):
+        k0, v0 = sw.initial()
+        for B in batches:
+            n_meas = max(10, (2_000_000 + 2 * B - 1) // (2 * B))
+            n_meas = min(n_meas, avail // B - 3)
+            g = Gpma.gpma_create(cfg.V, k0.contiguous(), v0.contiguous(), stream=s)
+            times = []
+            pos = 0
+            for it in range(3 + n_meas):
+                dk = sw.keys[pos:pos + B]
+                ik = sw.keys[sw.window + pos: sw.window + pos + B]
+                iv = sw.vals[sw.window + pos: sw.window + pos + B]
+                pos += B
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                e0.record(s)
+                g.gpma_update_batch(dk, None, 1, stream=s)
+                g.gpma_update_batch(ik, iv, 0, stream=s)
+                e1.record(s)
+                e1.synchronize()
+                if it >= 3:
+                    times.append(e0.elapsed_time(e1))
+            del g
+            t = np.array(times)
+            res.append({"batch": B, "slides": len(times), "updates_per_s": 2 * B / (t.mean() / 1e3),
+                        "ms_per_slide_mean": float(t.mean()), "ms_p50": float(np.percentile(t, 50)),
+                        "ms_p99": float(np.percentile(t, 99))})
+    return {"workload": "configs[1] pokec-shaped (V=1.6M, 15M-edge window)", "points": res}
 
 
 # ------------------------------------------------------------------ GPMA arm, N > 1

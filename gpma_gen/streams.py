@@ -223,6 +223,9 @@ def config_stream(cfg: int | StreamConfig, seed: int | None = None, device="cpu"
     sd = c.seed if seed is None else seed
     keys = make_stream(c.kind, c.V, c.E, sd, scale=c.scale, device=device)
     vals = edge_values(keys, sd)
+    if torch.device(device).type == "cuda":
+        # generated on torch's current stream; consumers may use other streams
+        torch.cuda.synchronize(device)
     return SlidingWindow(keys, vals, c.window, c.batch)
 
 
