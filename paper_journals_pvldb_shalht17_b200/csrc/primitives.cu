@@ -144,10 +144,10 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
   __shared__ T ws[SC_THREADS / 32];
   __shared__ T s_prefix;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  if (threadIdx.x == 0) s_tile = (uint32_t)atomicAdd(status, 1ull);  // status[0] = tile counter
+  if (threadIdx.x == 0) s_tile = status ? (uint32_t)atomicAdd(status, 1ull) : 0u;  // status[0] = tile counter
   __syncthreads();
   const uint32_t tile = s_tile;
-  volatile unsigned long long *st = status + 1;
+  volatile unsigned long long *st = status ? status + 1 : nullptr;   // null: single tile
   const uint64_t base = (uint64_t)tile * SC_TILE + (uint64_t)w * (32 * SC_ITEMS);
   T x[SC_ITEMS];
   T part = 0;
@@ -165,7 +165,7 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
     for (int k = 0; k < SC_THREADS / 32; ++k) agg += ws[k];
     const unsigned long long VMASK = (1ull << 62) - 1;
     T prefix = 0;
-    if (lane == 0) {
+    if (lane == 0 && st) {
       __threadfence();
       st[tile] = ((tile == 0 ? 2ull : 1ull) << 62) | ((unsigned long long)agg & VMASK);
     }
@@ -185,7 +185,7 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
       t -= 32;
     }
     if (lane == 0) {
-      if (tile) {
+      if (tile && st) {
         __threadfence();
         st[tile] = (2ull << 62) | ((unsigned long long)(prefix + agg) & VMASK);
       }
@@ -208,6 +208,10 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
 template <typename T>
 static void scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) {
   const uint64_t nt = (n + SC_TILE - 1) / SC_TILE > 0 ? (n + SC_TILE - 1) / SC_TILE : 1;
+  if (nt == 1) {                       // one tile: no look-back, no status reset
+    GP_LAUNCH(g, k_scan_lookback<T>, 1, SC_THREADS, 0, s, in, out, n, (unsigned long long *)nullptr);
+    return;
+  }
   ensure(g->b_scan, (nt + 1) * sizeof(unsigned long long), s);
   unsigned long long *status = (unsigned long long *)g->b_scan.p;
   cudaMemsetAsync(status, 0, (nt + 1) * sizeof(unsigned long long), s);
@@ -310,9 +314,49 @@ __global__ void __launch_bounds__(RS_THREADS) k_radix_scatter(
   }
 }
 
+// Small batches: one CTA sorts (key, arrival index) pairs with a bitonic network in shared
+// memory -- stable by construction (the index breaks ties) -- and gathers the values.  One
+// launch instead of 4 per radix pass.
+constexpr int SS_MAX = 2048;
+__global__ void __launch_bounds__(1024) k_small_sort(uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1,
+                                                     uint32_t n) {
+  __shared__ uint64_t sk[SS_MAX];
+  __shared__ uint32_t si[SS_MAX];
+  uint32_t np2 = 1;
+  while (np2 < n) np2 <<= 1;
+  for (uint32_t i = threadIdx.x; i < np2; i += blockDim.x) {
+    sk[i] = i < n ? k0[i] : ~0ull;
+    si[i] = i;
+  }
+  __syncthreads();
+  for (uint32_t size = 2; size <= np2; size <<= 1)
+    for (uint32_t stride = size >> 1; stride; stride >>= 1) {
+      for (uint32_t i = threadIdx.x; i < np2; i += blockDim.x) {
+        const uint32_t j = i ^ stride;
+        if (j > i) {
+          const bool up = (i & size) == 0;
+          const bool gt = sk[i] > sk[j] || (sk[i] == sk[j] && si[i] > si[j]);
+          if (gt == up) {
+            uint64_t tk = sk[i]; sk[i] = sk[j]; sk[j] = tk;
+            uint32_t ti = si[i]; si[i] = si[j]; si[j] = ti;
+          }
+        }
+      }
+      __syncthreads();
+    }
+  for (uint32_t i = threadIdx.x; i < n; i += blockDim.x) {
+    k1[i] = sk[i];
+    v1[i] = v0[si[i]];
+  }
+}
+
 int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1, uint64_t n,
                      const int *shifts, int nshift, cudaStream_t s) {
   if (n <= 1) return 0;
+  if (n <= (uint64_t)SS_MAX) {
+    GP_LAUNCH(g, k_small_sort, 1, 1024, 0, s, k0, v0, k1, v1, (uint32_t)n);
+    return 1;
+  }
   const uint32_t ntiles = (uint32_t)((n + RS_TILE - 1) / RS_TILE);
   const uint64_t hn = (uint64_t)ntiles * 256;
   ensure(g->b_hist, (hn + 1) * sizeof(uint32_t), s);

@@ -59,6 +59,7 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
                           uint32_t nleaves, uint32_t L, int op, int mode,
                           uint32_t *__restrict__ keep, uint32_t *__restrict__ tgt, Ctrl *c,
                           uint32_t *__restrict__ tmask, uint32_t *__restrict__ deg, uint32_t rb) {
+  if (c->err) return;                                // rejected batch: nothing may change
   uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
   uint32_t uniq = 0;
   if (i < n) {
@@ -115,7 +116,8 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
 __global__ void k_lazy_delete(const uint64_t *__restrict__ keys, uint64_t n, const uint64_t *__restrict__ key,
                               uint32_t *val, uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
                               uint32_t nleaves, uint32_t L, uint32_t *__restrict__ tmask,
-                              uint32_t *__restrict__ deg, uint32_t rb) {
+                              uint32_t *__restrict__ deg, uint32_t rb, const Ctrl *c) {
+  if (c->err) return;                                // rejected batch: nothing may change
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
        i += (uint64_t)gridDim.x * blockDim.x) {
     const uint64_t k = keys[i];
@@ -150,12 +152,15 @@ __global__ void k_lazy_delete(const uint64_t *__restrict__ keys, uint64_t n, con
 // index plus the live entries below it -- and writes the left-packed leaf back (a one-leaf
 // window has a single piece in the R7 split).  Rejected groups stay pending for level 1.
 __global__ void __launch_bounds__(256) k_level0(const uint64_t *__restrict__ pk, const uint32_t *__restrict__ pv,
-                                                const uint32_t *__restrict__ pt, uint64_t p, uint64_t *key,
+                                                const uint32_t *__restrict__ pt, const uint32_t *__restrict__ p_dev,
+                                                uint64_t *key,
                                                 uint32_t *val, uint32_t *__restrict__ cnt,
                                                 uint32_t *__restrict__ tmask, uint64_t *__restrict__ head,
                                                 uint64_t *__restrict__ row_offset, uint32_t rb, uint32_t L,
                                                 uint32_t bound, int op, uint32_t *__restrict__ keep,
                                                 uint2 *__restrict__ dirty, Ctrl *c) {
+  if (c->err) return;
+  const uint64_t p = *p_dev;                         // pending updates (device-side count)
   const int lane = threadIdx.x & 31;
   const uint32_t lt = (1u << lane) - 1u;
   const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
@@ -272,7 +277,8 @@ __global__ void k_compact_pending(const uint32_t *__restrict__ keep, const uint3
                                   uint64_t n, const uint64_t *__restrict__ ik,
                                   const uint32_t *__restrict__ iv, const uint32_t *__restrict__ it,
                                   uint64_t *__restrict__ ok, uint32_t *__restrict__ ov,
-                                  uint32_t *__restrict__ ot) {
+                                  uint32_t *__restrict__ ot, const Ctrl *c) {
+  if (c->err) return;
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
        i += (uint64_t)gridDim.x * blockDim.x) {
     if (keep[i]) {
@@ -971,7 +977,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   if (out->p_new && !resize_target) {
     GP_LAUNCH(g, k_compact_pending, grid_for(p), TB, 0, s, a.keep, a.kpos, p, a.pk, a.pv, a.pt,
               (uint64_t *)g->b_pk[cur ^ 1].p, (uint32_t *)g->b_pv[cur ^ 1].p,
-              (uint32_t *)g->b_pt[cur ^ 1].p);
+              (uint32_t *)g->b_pt[cur ^ 1].p, g->ctrl_d);
   }
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
@@ -1084,27 +1090,44 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   return recompute_heads(g, s);
 }
 
+__global__ void k_upd_summary(const uint32_t *__restrict__ pos, const uint32_t *__restrict__ kpos, uint64_t n,
+                              Ctrl *c) {
+  c->sum = pos[n];                                   // pending after the pre-pass
+  c->sum2 = kpos ? kpos[n] : 0;                      // pending after level 0
+}
+
+static gpma_status status_of(gpma *g) {
+  if (g->ctrl_h->err & 2u) return GPMA_ERR_RESERVED;
+  if (g->ctrl_h->err & 1u) return GPMA_ERR_RANGE;
+  return GPMA_OK;
+}
+
+// One batch.  Validation runs on the device and every mutating kernel bails out when it
+// flagged the batch, so the common insert path (sort -> pre-pass -> fused level 0) needs a
+// single host round trip; the generic levels >= 1 and the resize follow only when level 0
+// leaves updates pending.
 gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op,
                          cudaStream_t s) {
   gpma_status st;
   g->last = gpma_stats_t{};
   g->trace.clear();
   if (n == 0) return GPMA_OK;
-  // stage (host or device input) -- sort_unique copies into its own buffers anyway
   GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
   GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
   uint64_t *ik = (uint64_t *)g->b_stage[0].p;
   uint32_t *iv = (uint32_t *)g->b_stage[1].p;
   GP_CHECK(g, cudaMemcpyAsync(ik, keys, n * 8, cudaMemcpyDefault, s));
   if (op == GPMA_INSERT) GP_CHECK(g, cudaMemcpyAsync(iv, vals, n * 4, cudaMemcpyDefault, s));
-  if ((st = validate(g, ik, iv, n, op == GPMA_INSERT, s))) return st;
+  if ((st = zero_ctrl(g, s))) return st;
+  GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, ik, iv, n, g->V, g->rb, g->nr, op == GPMA_INSERT ? 1 : 0,
+            g->ctrl_d);
+  const uint64_t nl = g->cap / g->L;
   if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
-    const uint64_t nl0 = g->cap / g->L;
-    GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl0,
-              g->L, tmask_of(g), g->deg, g->rb);
+    GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
+              tmask_of(g), g->deg, g->rb, g->ctrl_d);
+    if ((st = read_ctrl(g, s))) return st;
     g->last.last_unique = n;   // not deduplicated: lazy deletes are idempotent
-    GP_CHECK(g, cudaGetLastError());
-    return GPMA_OK;
+    return status_of(g);
   }
   int which;
   uint64_t m;
@@ -1116,40 +1139,34 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   GP_CHECK(g, ensure(g->b_tgt, (n + 1) * 4, s));
   if ((st = level_buffers(g, n, s))) return st;
   uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p, *tgt = (uint32_t *)g->b_tgt.p;
-  if ((st = zero_ctrl(g, s))) return st;
-  const uint64_t nl = g->cap / g->L;
-  GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt,
-            g->head, (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb);
+  GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt, g->head,
+            (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb);
   scan_u32(g, keep, pos, n, s);
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, pos + n, 4, cudaMemcpyDeviceToHost, s));
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->nunique, &g->ctrl_d->nunique, 8, cudaMemcpyDeviceToHost, s));
-  GP_CHECK(g, cudaStreamSynchronize(s));
-  uint64_t p = (uint32_t)g->ctrl_h->sum2;
+  GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, tgt, (uint64_t *)g->b_pk[0].p,
+            (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p, g->ctrl_d);
+  uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
+  const bool fused = !g->trace_on;   // the per-level trace needs the generic level-0 step
+  if (fused) {
+    // level 0 fused: one warp per leaf group, sized by n, counts read on the device
+    GP_CHECK(g, cudaMemsetAsync(keep2, 0, (n + 1) * 4, s));
+    const uint32_t bound = (uint32_t)(op == GPMA_INSERT ? g->tmax[0] : g->tmin[0]);
+    GP_LAUNCH(g, k_level0, grid_for((n + 31) / 32 * 32), 256, 0, s, (const uint64_t *)g->b_pk[0].p,
+              (const uint32_t *)g->b_pv[0].p, (const uint32_t *)g->b_pt[0].p, pos + n, g->key, g->val, g->cnt,
+              tmask_of(g), g->head, g->row_offset, g->rb, g->L, bound, op, keep2, (uint2 *)g->b_dirty.p,
+              g->ctrl_d);
+    scan_u32(g, keep2, kpos, n, s);
+  }
+  GP_LAUNCH(g, k_upd_summary, 1, 1, 0, s, pos, fused ? kpos : nullptr, n, g->ctrl_d);
+  if ((st = read_ctrl(g, s))) return st;             // the one host round trip of the batch
+  if ((st = status_of(g))) return st;
+  uint64_t p = (uint32_t)g->ctrl_h->sum;
   g->last.last_unique = g->ctrl_h->nunique;
   g->last.last_pending = p;
   if (p == 0) return GPMA_OK;
   int cur = 0;
-  GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, tgt,
-            (uint64_t *)g->b_pk[0].p, (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p);
   uint64_t dirty_base = 0;
   uint32_t lvl = 0;
-  if (!g->trace_on) {
-    // level 0 fused: one warp per leaf group (the generic step below serves levels >= 1,
-    // and level 0 too when the per-level trace is requested)
-    GP_CHECK(g, cudaMemsetAsync(&g->ctrl_d->ndirty, 0, 16, s));   // ndirty + sum
-    GP_CHECK(g, cudaMemsetAsync(&g->ctrl_d->windows_rewritten, 0, 8, s));
-    uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
-    const uint32_t bound = (uint32_t)(op == GPMA_INSERT ? g->tmax[0] : g->tmin[0]);
-    GP_LAUNCH(g, k_level0, grid_for((p + 31) / 32 * 32), 256, 0, s, (const uint64_t *)g->b_pk[0].p,
-              (const uint32_t *)g->b_pv[0].p, (const uint32_t *)g->b_pt[0].p, p, g->key, g->val, g->cnt,
-              tmask_of(g), g->head, g->row_offset, g->rb, g->L, bound, op, keep2, (uint2 *)g->b_dirty.p,
-              g->ctrl_d);
-    scan_u32(g, keep2, kpos, p, s);
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, kpos + p, 4, cudaMemcpyDeviceToHost, s));
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->ndirty, &g->ctrl_d->ndirty, 8, cudaMemcpyDeviceToHost, s));
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->windows_rewritten, &g->ctrl_d->windows_rewritten, 8,
-                                cudaMemcpyDeviceToHost, s));
-    GP_CHECK(g, cudaStreamSynchronize(s));
+  if (fused) {
     const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
     dirty_base = g->ctrl_h->ndirty;
     g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;
@@ -1157,7 +1174,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
     if (p_new) {
       GP_LAUNCH(g, k_compact_pending, grid_for(p), TB, 0, s, keep2, kpos, p, (const uint64_t *)g->b_pk[0].p,
                 (const uint32_t *)g->b_pv[0].p, (const uint32_t *)g->b_pt[0].p, (uint64_t *)g->b_pk[1].p,
-                (uint32_t *)g->b_pv[1].p, (uint32_t *)g->b_pt[1].p);
+                (uint32_t *)g->b_pv[1].p, (uint32_t *)g->b_pt[1].p, g->ctrl_d);
       cur = 1;
       g->last.last_top_level = 1;
     }
@@ -1176,8 +1193,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   }
   if (p > 0) {
     g->last.last_top_level = g->h + 1;
-    if ((st = resize(g, cur, p, op, s, &dirty_base))) return st;
-    return GPMA_OK;
+    return resize(g, cur, p, op, s, &dirty_base);
   }
   if (dirty_base) {
     GP_LAUNCH(g, k_heads_dirty, grid_for(dirty_base * 32), TB, 0, s, g->key, g->head, g->L, nl,
