@@ -1,0 +1,110 @@
+"""Degenerate and extreme inputs: the CUDA path must equal the oracle bit for bit."""
+import numpy as np
+import pytest
+import torch
+
+import oracle as O
+from tests.brute import Replay
+from tests.gpu_helpers import DEV, assert_same_csr, assert_same_layout, gpu_bfs, gpu_cc, keys_t, vals_t
+
+pytestmark = pytest.mark.gpu
+
+
+def _pair(V, keys, vals, **kw):
+    from paper_journals_pvldb_shalht17_b200 import Gpma
+    mode = kw.pop("delete_mode", 0)
+    L = kw.pop("leaf_slots", 0)
+    bp = kw.pop("thresholds_bp", None)
+    g = Gpma.gpma_create(V, keys_t(keys) if len(keys) else None, vals_t(vals) if len(keys) else None,
+                         delete_mode=mode, leaf_slots=L, thresholds_bp=bp)
+    o = O.Oracle(V, keys, vals, delete_mode=mode, leaf_slots=L)
+    if bp:
+        O.lib().orc_set_thresholds_bp(o._h, *bp)
+    return g, o
+
+
+def _apply(g, o, keys, vals=None, op=0):
+    if op == 0:
+        g.insert(keys_t(keys), vals_t(vals))
+        o.insert(keys, vals)
+    else:
+        g.delete(keys_t(keys))
+        o.delete(keys)
+    assert_same_layout(g, o)
+
+
+def test_single_vertex_self_loop():
+    g, o = _pair(1, [], [])
+    _apply(g, o, [0], [5])
+    assert gpu_bfs(g, 0).tolist() == [0] and gpu_cc(g).tolist() == [0]
+    _apply(g, o, [0], op=1)
+    _apply(g, o, [0], [6])
+    assert_same_csr(g, o)
+
+
+def test_extreme_ids_and_values():
+    V = (1 << 20) + 3
+    top = V - 1
+    keys = [(top << 32) | top, (top << 32), top, 0]
+    vals = [0, 0x7FFFFFFF, 0xFFFFFFFE, 1]
+    g, o = _pair(V, keys, vals)
+    _apply(g, o, [(top << 32) | (top - 1), (1 << 32) | top], [0xFFFFFFFE, 3])
+    _apply(g, o, [(top << 32) | top], op=1)
+    assert_same_csr(g, o)
+
+
+@pytest.mark.parametrize("mode", [0, 1])
+def test_all_duplicates_and_delete_everything(mode):
+    V = 64
+    g, o = _pair(V, [], [], delete_mode=mode)
+    k = (5 << 32) | 7
+    _apply(g, o, [k] * 3000, list(range(3000)))                  # radix-sort path, one key
+    rng = np.random.default_rng(2)
+    ks = list({int(a) << 32 | int(b) for a, b in zip(rng.integers(0, V, 3000), rng.integers(0, V, 3000))})
+    _apply(g, o, ks, [1] * len(ks))
+    _apply(g, o, ks + [k], op=1)                                 # the store is empty again
+    assert g.gpma_stats()["live_edges"] == 0
+    _apply(g, o, ks[:100], [2] * 100)                            # re-insert (revive in lazy mode)
+    assert_same_csr(g, o)
+
+
+@pytest.mark.parametrize("L", [4, 8, 32])
+def test_leaf_size_overrides(L):
+    rng = np.random.default_rng(L)
+    V = 300
+    keys = [int(a) << 32 | int(b) for a, b in zip(rng.integers(0, V, 2000), rng.integers(0, V, 2000))]
+    g, o = _pair(V, keys, [1] * len(keys), leaf_slots=L)
+    ref = Replay(V, keys, [1] * len(keys))
+    for step in range(12):
+        b = int(rng.integers(1, 3000))
+        ks = [int(a) << 32 | int(c) for a, c in zip(rng.integers(0, V, b), rng.integers(0, V, b))]
+        if step % 3 == 2:
+            _apply(g, o, ks, op=1)
+            ref.delete(ks)
+        else:
+            vs = rng.integers(0, 1 << 31, len(ks)).tolist()
+            _apply(g, o, ks, vs)
+            ref.insert(ks, vs)
+    assert g.gpma_stats()["leaf_slots"] == L
+    assert_same_csr(g, o)
+
+
+def test_threshold_overrides():
+    rng = np.random.default_rng(9)
+    V = 200
+    bp = (1500, 3000, 7000, 6000)                                # tighter bounds: more climbs/resizes
+    keys = [int(a) << 32 | int(b) for a, b in zip(rng.integers(0, V, 500), rng.integers(0, V, 500))]
+    g, o = _pair(V, keys, [0] * 500, thresholds_bp=bp, delete_mode=1)
+    for step in range(15):
+        ks = [int(a) << 32 | int(b) for a, b in zip(rng.integers(0, V, 400), rng.integers(0, V, 400))]
+        _apply(g, o, ks, [step] * len(ks), op=step % 2)
+
+
+def test_halving_down_to_minimum_capacity():
+    V = 4
+    keys = [(a << 32) | b for a in range(V) for b in range(V)]
+    g, o = _pair(V, keys, [1] * len(keys), delete_mode=1)
+    for k in keys:                                               # one at a time: many halvings
+        _apply(g, o, [k], op=1)
+    st = g.gpma_stats()
+    assert st["capacity"] == o.capacity and st["live_edges"] == 0
