@@ -66,7 +66,9 @@ typedef struct {
   uint16_t rho_leaf_bp, rho_root_bp, tau_leaf_bp, tau_root_bp; /* R4, basis points:
                                  800, 4000, 9200, 8000 = Fig. 3           */
   uint16_t init_density_bp;   /* R15: 6000                                            */
-  uint16_t reserved0;
+  uint16_t algorithm;         /* insertion: 0 = GPMA+ segment-oriented (Alg. 4, default);
+                                 1 = GPMA lock-based (Alg. 1) with deterministic
+                                 lock arbitration (the smallest key wins a segment)       */
   uint32_t delete_mode;       /* gpma_delete_mode                                     */
   uint32_t row_begin, row_end;/* shard (R24): the store holds the rows
                                  (sources) [row_begin, row_end) only -- guards, row
@@ -90,6 +92,7 @@ typedef struct {
   uint64_t last_windows_rewritten;
   uint32_t last_top_level;    /* highest level reached (h+1 = resized)                */
   uint32_t last_resized;
+  uint64_t last_rounds;       /* GPMA (algorithm 1): retry rounds of the last insert    */
 } gpma_stats_t;
 
 /* Fill *cfg with the defaults above. */

@@ -62,6 +62,8 @@ def lib():
             "orc_leaf_rule": (u32, [u64]),
             "orc_set_thresholds_bp": (None, [P, u32, u32, u32, u32]),
             "orc_bfs_csr": (None, [u32, P, P, u32, P]),
+            "orc_set_algorithm": (None, [P, i32]),
+            "orc_rounds_last": (u64, [P]),
             "orc_cc_csr": (None, [u32, P, P, P]),
             "orc_pagerank_csr": (i32, [u32, P, P, P, i32, C.c_double, C.c_double, i32]),
         }
@@ -117,7 +119,7 @@ class Oracle:
     """One sequential GPMA+ store."""
 
     def __init__(self, V: int, keys=(), vals=(), *, leaf_slots: int = 0, capacity: int = 0,
-                 delete_mode: int = LAZY, rows=None, _raw=None):
+                 delete_mode: int = LAZY, rows=None, algorithm: int = 0, _raw=None):
         st = C.c_int(0)
         if _raw is not None:
             cap, L, rk, rv = _raw
@@ -131,12 +133,18 @@ class Oracle:
         if st.value != OK:
             raise OracleError(st.value)
         self.V = V
+        lib().orc_set_algorithm(self._h, algorithm)
         self.rb, self.nr = (rows[0], rows[1] - rows[0]) if rows is not None and rows[1] > rows[0] else (0, V)
 
     @classmethod
-    def raw(cls, V, cap, L, keys, vals=None, delete_mode=LAZY):
+    def raw(cls, V, cap, L, keys, vals=None, delete_mode=LAZY, algorithm=0):
         vals = np.zeros(cap, np.uint32) if vals is None else vals
-        return cls(V, _raw=(cap, L, keys, vals), delete_mode=delete_mode)
+        return cls(V, _raw=(cap, L, keys, vals), delete_mode=delete_mode, algorithm=algorithm)
+
+    @property
+    def rounds(self) -> int:
+        """GPMA (Alg. 1): retry rounds of the last insert batch."""
+        return int(lib().orc_rounds_last(self._h))
 
     def __del__(self):
         if getattr(self, "_h", None):

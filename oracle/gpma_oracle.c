@@ -55,6 +55,8 @@ typedef struct orc {
   trace_t *trace; uint64_t ntrace, trace_cap;
   uint64_t slots_rewritten, windows_rewritten, top_level, pending_after_prepass;
   uint64_t resizes, resizes_last;
+  int algorithm;       /* 0 = GPMA+ (Alg. 4), 1 = GPMA lock-based (Alg. 1)            */
+  uint64_t rounds_last;/* GPMA: retry rounds of the last batch                        */
 } orc_t;
 
 /* ---------------------------------------------------------------- thresholds */
@@ -357,6 +359,107 @@ static int resize(orc_t *o, const upd_t *P, uint64_t np, int op) {
   return ORC_OK;
 }
 
+/* Root doubling of GPMA (Alg. 1 l.20 "double the space of the root segment"): all
+ * live entries re-dispatched evenly over twice the capacity (R7); nothing is inserted. */
+static int double_root(orc_t *o) {
+  uint64_t nlive = 0, s;
+  uint64_t *lk, *k2; uint32_t *lv, *v2;
+  for (s = 0; s < o->cap; s++) nlive += is_live(o, s);
+  lk = (uint64_t *)malloc(sizeof(uint64_t) * (nlive ? nlive : 1));
+  lv = (uint32_t *)malloc(sizeof(uint32_t) * (nlive ? nlive : 1));
+  collect_live(o, 0, o->cap, lk, lv);
+  k2 = (uint64_t *)malloc(sizeof(uint64_t) * o->cap * 2);
+  v2 = (uint32_t *)malloc(sizeof(uint32_t) * o->cap * 2);
+  free(o->key); free(o->val);
+  o->key = k2; o->val = v2;
+  set_geometry(o, o->cap * 2);
+  redispatch(o, 0, o->cap / o->L, lk, lv, nlive);
+  o->resizes++; o->resizes_last++;
+  o->slots_rewritten += o->cap;
+  o->windows_rewritten += 1;
+  free(lk); free(lv);
+  return ORC_OK;
+}
+
+static int cmp_upd(const void *a, const void *b) {
+  const upd_t *x = (const upd_t *)a, *y = (const upd_t *)b;
+  return x->key < y->key ? -1 : (x->key > y->key);
+}
+
+/* GPMA concurrent insertion (Alg. 1; Ex. 2) with deterministic lock
+ * arbitration: every insertion searches its leaf, then the rounds climb level by level
+ * ("all threads are synchronized after updating all segments located at the same tree
+ * height").  At each level the insertions that reach the same segment compete for
+ * its lock; the one with the smallest key wins (the paper leaves the winner unspecified --
+ * "Assuming Insertion-1 succeeds") and the others abort until the next round
+ * (l.11-12).  A winner whose segment can take one more entry (count + 1 <= max_i, R5) merges
+ * and re-dispatches it (l.16-17); otherwise it climbs (l.13-14).  As for GPMA+ (R6), the root
+ * is tested too; a winner the root cannot take doubles it (l.20) and retries next round.  Rounds repeat until every insertion
+ * took effect (l.2). */
+static int gpma_lock_insert(orc_t *o, upd_t *P, uint64_t np) {
+  upd_t *A = (upd_t *)malloc(sizeof(upd_t) * (np ? np : 1));
+  upd_t *W = (upd_t *)malloc(sizeof(upd_t) * (np ? np : 1));
+  uint64_t *wk = NULL; uint32_t *wv = NULL; uint64_t wcap = 0;
+  o->rounds_last = 0;
+  while (np > 0) {
+    uint64_t na = 0, nw, j, nne;
+    uint32_t i;
+    uint64_t *ne = nonempty_leaves(o, &nne);
+    o->rounds_last++;
+    for (j = 0; j < np; j++) P[j].leaf = target_leaf(o, ne, nne, P[j].key);   /* l.4 */
+    free(ne);
+    memcpy(W, P, sizeof(upd_t) * np);
+    nw = np;
+    for (i = 0; i <= o->h && nw > 0; i++) {           /* up to the root, tested too (R6) */
+      uint64_t nk = 0, g0 = 0;
+      while (g0 < nw) {
+        uint64_t seg = W[g0].leaf >> i, g1 = g0 + 1, s0, s1, n = 0, s;
+        while (g1 < nw && (W[g1].leaf >> i) == seg) A[na++] = W[g1++];   /* lose the lock: abort */
+        s0 = (seg << i) * o->L; s1 = s0 + ((uint64_t)o->L << i);
+        for (s = s0; s < s1; s++) n += is_live(o, s);
+        if (n + 1 <= o->tmax[i]) {                    /* l.13 test fails -> insert (l.16-17) */
+          uint64_t a = 0, c = 0;
+          uint64_t *lk = (uint64_t *)malloc(sizeof(uint64_t) * (n ? n : 1));
+          uint32_t *lv = (uint32_t *)malloc(sizeof(uint32_t) * (n ? n : 1));
+          int placed = 0;
+          collect_live(o, s0, s1, lk, lv);
+          if (n + 1 > wcap) {
+            wcap = n + 1;
+            wk = (uint64_t *)realloc(wk, sizeof(uint64_t) * wcap);
+            wv = (uint32_t *)realloc(wv, sizeof(uint32_t) * wcap);
+          }
+          for (a = 0; a < n; a++) {
+            if (!placed && W[g0].key < lk[a]) { wk[c] = W[g0].key; wv[c] = W[g0].val; c++; placed = 1; }
+            wk[c] = lk[a]; wv[c] = lv[a]; c++;
+          }
+          if (!placed) { wk[c] = W[g0].key; wv[c] = W[g0].val; c++; }
+          free(lk); free(lv);
+          redispatch(o, seg << i, 1ull << i, wk, wv, c);
+          o->slots_rewritten += s1 - s0;
+          o->windows_rewritten += 1;
+        } else {
+          W[nk++] = W[g0];                            /* climb to the parent (l.14) */
+        }
+        g0 = g1;
+      }
+      nw = nk;
+      if (i > o->top_level) o->top_level = i;
+    }
+    if (nw > 0) {                                     /* reached the root: double (l.20) */
+      double_root(o);
+      for (j = 0; j < nw; j++) A[na++] = W[j];
+    }
+    qsort(A, na, sizeof(upd_t), cmp_upd);
+    memcpy(P, A, sizeof(upd_t) * na);
+    np = na;
+  }
+  free(A); free(W); free(wk); free(wv);
+  return ORC_OK;
+}
+
+void orc_set_algorithm(orc_t *o, int algorithm) { o->algorithm = algorithm; }
+uint64_t orc_rounds_last(const orc_t *o) { return o->rounds_last; }
+
 /* GpmaPlusInsertion (Alg. 4) and its dual for strict deletions over the
  * pending list P (sorted by key, with leaf targets). */
 static int level_loop(orc_t *o, upd_t *P, uint64_t np, int op) {
@@ -455,7 +558,8 @@ int orc_update(orc_t *o, const uint64_t *keys, const uint32_t *vals, uint64_t n,
   }
   free(ne); free(u);
   o->pending_after_prepass = np;
-  st = np ? level_loop(o, P, np, op) : ORC_OK;
+  if (np && op == ORC_INSERT && o->algorithm == 1) st = gpma_lock_insert(o, P, np);
+  else st = np ? level_loop(o, P, np, op) : ORC_OK;
   free(P);
   return st;
 }

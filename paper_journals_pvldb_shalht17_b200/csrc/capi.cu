@@ -80,7 +80,8 @@ gpma_status apply_config(gpma *g, const gpma_config *cfg, uint32_t *leaf, uint64
   }
   if (c.leaf_slots && (c.leaf_slots < 4 || c.leaf_slots > 32 || (c.leaf_slots & (c.leaf_slots - 1))))
     return GPMA_ERR_INVALID_ARG;
-  if (c.delete_mode > 1) return GPMA_ERR_INVALID_ARG;
+  if (c.delete_mode > 1 || c.algorithm > 1) return GPMA_ERR_INVALID_ARG;
+  g->algorithm = c.algorithm;
   if (c.rho_leaf_bp > 10000 || c.rho_root_bp > 10000 || c.tau_leaf_bp > 10000 || c.tau_root_bp > 10000 ||
       c.init_density_bp == 0 || c.init_density_bp > 10000)
     return GPMA_ERR_INVALID_ARG;

@@ -1090,10 +1090,184 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   return recompute_heads(g, s);
 }
 
+// ---- GPMA lock-based insertion (Alg. 1) -----------------------------------------------
+__global__ void k_count_leaf_live(const uint32_t *__restrict__ cnt, uint64_t nl, uint64_t *__restrict__ out) {
+  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nl;
+       l += (uint64_t)gridDim.x * blockDim.x)
+    out[l] = cnt[l];
+}
+
+__global__ void k_relocate(const uint64_t *__restrict__ pk, uint64_t p, const uint64_t *__restrict__ head,
+                           uint32_t nleaves, uint32_t *__restrict__ pt) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < p;
+       j += (uint64_t)gridDim.x * blockDim.x)
+    pt[j] = locate_leaf(head, nleaves, pk[j]);
+}
+
+// lock arbitration at one level: the first (smallest key) insertion of every segment keeps
+// going (winner list), the others abort to the next round (loser list, appended at `na`)
+__global__ void k_lock_split(const uint64_t *__restrict__ pk, const uint32_t *__restrict__ pv,
+                             const uint32_t *__restrict__ pt, const uint32_t *__restrict__ hf,
+                             const uint32_t *__restrict__ widx, uint64_t p, uint64_t *__restrict__ wk,
+                             uint32_t *__restrict__ wv, uint32_t *__restrict__ wt, uint64_t *__restrict__ ak,
+                             uint32_t *__restrict__ av, uint64_t na) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < p;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    if (hf[j]) {
+      const uint32_t d = widx[j];
+      wk[d] = pk[j];
+      wv[d] = pv[j];
+      wt[d] = pt[j];
+    } else {
+      const uint64_t d = na + j - widx[j];
+      ak[d] = pk[j];
+      av[d] = pv[j];
+    }
+  }
+}
+
+__global__ void k_append_kv(const uint64_t *__restrict__ k, const uint32_t *__restrict__ v, uint64_t n,
+                            uint64_t *__restrict__ ak, uint32_t *__restrict__ av, uint64_t na) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < n;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    ak[na + j] = k[j];
+    av[na + j] = v[j];
+  }
+}
+
+// dense list of every live entry (guards included, tombstones dropped), in key order
+__global__ void k_gather_live(const uint64_t *__restrict__ key, const uint32_t *__restrict__ val, uint32_t L,
+                              uint64_t cap, const uint64_t *__restrict__ lbase, uint64_t *__restrict__ wk,
+                              uint32_t *__restrict__ wv) {
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint32_t leafmask = (L == 32 ? 0xffffffffu : ((1u << L) - 1u) << (lane & ~(L - 1)));
+  const uint64_t capr = (cap + 31) & ~31ull;
+  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < capr;
+       s += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t k = KEY_NONE;
+    uint32_t v = 0;
+    if (s < cap) {
+      k = key[s];
+      v = val[s];
+    }
+    const bool live = s < cap && k != KEY_NONE && v != VAL_TOMB;
+    const uint32_t bal = __ballot_sync(0xffffffffu, live);
+    if (live) {
+      const uint64_t d = lbase[s / L] + __popc(bal & leafmask & lt);
+      wk[d] = k;
+      wv[d] = v;
+    }
+  }
+}
+
+// Alg. 1 l.20: double the space of the root segment -- all live entries re-dispatched evenly
+// over twice the capacity (R7); the insertion that reached the root retries.
+static gpma_status double_root(gpma *g, cudaStream_t s) {
+  gpma_status st;
+  const uint64_t nl = g->cap / g->L, cap2 = g->cap * 2;
+  GP_CHECK(g, ensure(g->b_lpre, (nl + 1) * 8, s));
+  uint64_t *lb = (uint64_t *)g->b_lpre.p;
+  GP_LAUNCH(g, k_count_leaf_live, grid_for(nl), TB, 0, s, g->cnt, nl, lb);
+  scan_u64(g, lb, lb, nl, s);
+  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, lb + nl, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  const uint64_t N = g->ctrl_h->sum;
+  GP_CHECK(g, ensure(g->b_wk, std::max<uint64_t>(N, 1) * 8, s));
+  GP_CHECK(g, ensure(g->b_wv, std::max<uint64_t>(N, 1) * 4, s));
+  GP_LAUNCH(g, k_gather_live, grid_for(g->cap), TB, 0, s, g->key, g->val, g->L, g->cap, lb,
+            (uint64_t *)g->b_wk.p, (uint32_t *)g->b_wv.p);
+  uint64_t *nk;
+  uint32_t *nv, *ncnt;
+  uint64_t *nhead;
+  if ((st = alloc_store(g, cap2, &nk, &nv, &ncnt, &nhead, s))) return st;
+  GP_LAUNCH(g, k_layout_even, grid_for(cap2), TB, 0, s, (const uint64_t *)g->b_wk.p, (const uint32_t *)g->b_wv.p,
+            N, nk, nv, ncnt, g->row_offset, g->L, cap2 / g->L, g->rb);
+  cudaFreeAsync(g->key, s);
+  cudaFreeAsync(g->val, s);
+  cudaFreeAsync(g->cnt, s);
+  cudaFreeAsync(g->head, s);
+  g->key = nk;
+  g->val = nv;
+  g->cnt = ncnt;
+  g->head = nhead;
+  g->resizes++;
+  g->last.last_resized = 1;
+  set_geometry(g, cap2);
+  g->last.last_slots_rewritten += cap2;
+  g->last.last_windows_rewritten += 1;
+  return recompute_heads(g, s);
+}
+
 __global__ void k_upd_summary(const uint32_t *__restrict__ pos, const uint32_t *__restrict__ kpos, uint64_t n,
                               Ctrl *c) {
   c->sum = pos[n];                                   // pending after the pre-pass
   c->sum2 = kpos ? kpos[n] : 0;                      // pending after level 0
+}
+
+// GPMA concurrent insertion (Alg. 1): rounds of level-synchronous climbs with one
+// lock per segment.  Lock arbitration is deterministic -- the first (smallest-key) insertion
+// that reaches a segment wins it, the others abort to the next round -- so the layout is
+// reproducible (the oracle follows the same rule).  Winners test count + 1 <= max_i and are
+// merged by the generic level step; a winner that reaches the root doubles it (l.20).
+static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
+  gpma_status st;
+  GP_CHECK(g, ensure(g->b_stage[2], (p + 1) * 8, s));
+  GP_CHECK(g, ensure(g->b_stage[3], (p + 1) * 4, s));
+  uint64_t *ak = (uint64_t *)g->b_stage[2].p;
+  uint32_t *av = (uint32_t *)g->b_stage[3].p;
+  uint64_t rounds = 0;
+  while (p > 0) {
+    ++rounds;
+    int cur = 0;
+    const uint64_t nl = g->cap / g->L;
+    GP_LAUNCH(g, k_relocate, grid_for(p), TB, 0, s, (const uint64_t *)g->b_pk[0].p, p, g->head, (uint32_t)nl,
+              (uint32_t *)g->b_pt[0].p);
+    uint64_t na = 0, nw = p, dirty_base = 0;
+    for (uint32_t lvl = 0; lvl <= g->h && nw > 0; ++lvl) {   // the root is tested too (R6)
+      Lvl a = make_lvl(g, cur, nw, lvl, GPMA_INSERT);
+      GP_LAUNCH(g, k_lvl_flags, grid_for(nw), TB, 0, s, a);
+      scan_u32(g, a.hf, a.widx, nw, s);
+      GP_LAUNCH(g, k_lock_split, grid_for(nw), TB, 0, s, a.pk, a.pv, a.pt, a.hf, a.widx, nw,
+                (uint64_t *)g->b_pk[cur ^ 1].p, (uint32_t *)g->b_pv[cur ^ 1].p, (uint32_t *)g->b_pt[cur ^ 1].p, ak,
+                av, na);
+      GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, a.widx + nw, 4, cudaMemcpyDeviceToHost, s));
+      GP_CHECK(g, cudaStreamSynchronize(s));
+      const uint64_t q = (uint32_t)g->ctrl_h->sum;      // lock winners at this level
+      na += nw - q;
+      cur ^= 1;
+      nw = q;
+      Lvl b = make_lvl(g, cur, nw, lvl, GPMA_INSERT);
+      LevelOut lo{};
+      if ((st = level_step(g, b, cur, &lo, &dirty_base, s, false, 0, nullptr, nullptr, nullptr))) return st;
+      g->last.last_slots_rewritten += lo.nacc * ((uint64_t)g->L << lvl);
+      g->last.last_windows_rewritten += lo.nacc;
+      if (lvl > g->last.last_top_level) g->last.last_top_level = lvl;
+      if (lo.p_new) cur ^= 1;
+      nw = lo.p_new;
+    }
+    if (nw > 0) {                                       // the root could not take it: double, retry
+      GP_LAUNCH(g, k_append_kv, grid_for(nw), TB, 0, s, (const uint64_t *)g->b_pk[cur].p,
+                (const uint32_t *)g->b_pv[cur].p, nw, ak, av, na);
+      na += nw;
+      g->last.last_top_level = g->h + 1;
+      if ((st = double_root(g, s))) return st;
+    } else if (dirty_base) {
+      GP_LAUNCH(g, k_heads_dirty, grid_for(dirty_base * 32), TB, 0, s, g->key, g->head, g->L, nl,
+                (const uint2 *)g->b_dirty.p, dirty_base);
+    }
+    if (na) {                                           // the aborted insertions, sorted again
+      int which;
+      uint64_t m;
+      if ((st = sort_unique(g, ak, av, na, &m, false, &which, s))) return st;
+      GP_CHECK(g, cudaMemcpyAsync(g->b_pk[0].p, g->b_sk[which].p, na * 8, cudaMemcpyDeviceToDevice, s));
+      GP_CHECK(g, cudaMemcpyAsync(g->b_pv[0].p, g->b_sv[which].p, na * 4, cudaMemcpyDeviceToDevice, s));
+    }
+    p = na;
+  }
+  g->last.last_rounds = rounds;
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
 }
 
 static gpma_status status_of(gpma *g) {
@@ -1145,7 +1319,8 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, tgt, (uint64_t *)g->b_pk[0].p,
             (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p, g->ctrl_d);
   uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
-  const bool fused = !g->trace_on;   // the per-level trace needs the generic level-0 step
+  const bool lock = op == GPMA_INSERT && g->algorithm == 1;   // GPMA (Alg. 1) instead of GPMA+
+  const bool fused = !g->trace_on && !lock;   // the per-level trace needs the generic level-0 step
   if (fused) {
     // level 0 fused: one warp per leaf group, sized by n, counts read on the device
     GP_CHECK(g, cudaMemsetAsync(keep2, 0, (n + 1) * 4, s));
@@ -1163,6 +1338,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   g->last.last_unique = g->ctrl_h->nunique;
   g->last.last_pending = p;
   if (p == 0) return GPMA_OK;
+  if (lock) return gpma_lock_insert(g, p, s);
   int cur = 0;
   uint64_t dirty_base = 0;
   uint32_t lvl = 0;

@@ -33,7 +33,7 @@ class GpmaError(RuntimeError):
 class gpma_config(C.Structure):
     _fields_ = [("struct_size", C.c_uint32), ("leaf_slots", C.c_uint32), ("initial_capacity", C.c_uint64),
                 ("rho_leaf_bp", C.c_uint16), ("rho_root_bp", C.c_uint16), ("tau_leaf_bp", C.c_uint16),
-                ("tau_root_bp", C.c_uint16), ("init_density_bp", C.c_uint16), ("reserved0", C.c_uint16),
+                ("tau_root_bp", C.c_uint16), ("init_density_bp", C.c_uint16), ("algorithm", C.c_uint16),
                 ("delete_mode", C.c_uint32), ("row_begin", C.c_uint32), ("row_end", C.c_uint32)]
 
 
@@ -43,7 +43,7 @@ class gpma_stats_t(C.Structure):
                 ("tombstones", C.c_uint64), ("resizes", C.c_uint64), ("last_unique", C.c_uint64),
                 ("last_pending", C.c_uint64), ("last_slots_rewritten", C.c_uint64),
                 ("last_windows_rewritten", C.c_uint64), ("last_top_level", C.c_uint32),
-                ("last_resized", C.c_uint32)]
+                ("last_resized", C.c_uint32), ("last_rounds", C.c_uint64)]
 
 
 _lib = None
@@ -147,9 +147,10 @@ class Gpma:
     @classmethod
     def gpma_create(cls, num_vertices: int, init_keys=None, init_vals=None, *, leaf_slots: int = 0,
                     initial_capacity: int = 0, delete_mode: int = DELETE_LAZY, thresholds_bp=None,
-                    init_density_bp: int = 6000, rows=None, stream=None) -> "Gpma":
+                    init_density_bp: int = 6000, rows=None, algorithm: int = 0, stream=None) -> "Gpma":
         cfg = gpma_config()
         lib().gpma_config_default(C.byref(cfg))
+        cfg.algorithm = algorithm
         if rows is not None:
             cfg.row_begin, cfg.row_end = rows
         cfg.leaf_slots = leaf_slots
@@ -168,10 +169,11 @@ class Gpma:
 
     @classmethod
     def gpma_create_raw(cls, num_vertices: int, capacity: int, leaf_slots: int, keys, vals, *,
-                        delete_mode: int = DELETE_LAZY, stream=None) -> "Gpma":
+                        delete_mode: int = DELETE_LAZY, algorithm: int = 0, stream=None) -> "Gpma":
         cfg = gpma_config()
         lib().gpma_config_default(C.byref(cfg))
         cfg.delete_mode = delete_mode
+        cfg.algorithm = algorithm
         h = C.c_void_p()
         st = lib().gpma_create_raw(num_vertices, capacity, leaf_slots, _ptr(keys), _ptr(vals), C.byref(cfg),
                                    _stream(stream), C.byref(h))

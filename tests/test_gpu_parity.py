@@ -259,3 +259,50 @@ def test_sorted_stream_hot_window():
         g.insert(keys_t(ks), vals_t([b] * 3000))
         o.insert(ks, [b] * 3000)
         assert_same_layout(g, o, what=f"hot batch {b}")
+
+
+def test_gpma_lock_example2_on_gpu(golden):
+    """NEXT-2: GPMA (Alg. 1) on the GPU, Ex. 2 batch: same rounds and layout as the oracle."""
+    g2 = golden("ex2_gpma_lock.json")
+    raw = fig3_layout()
+    g = Gpma.gpma_create_raw(64, 32, 4, raw.to(DEV), torch.zeros(32, dtype=torch.int32, device=DEV), algorithm=1)
+    o = O.Oracle.raw(64, 32, 4, raw, algorithm=1)
+    g.insert(keys_t(g2["batch"]), vals_t([0] * 5))
+    o.insert(g2["batch"], [0] * 5)
+    assert g.gpma_stats()["last_rounds"] == o.rounds == g2["rounds"]
+    assert_same_layout(g, o, guards=False, what="ex2")
+
+
+@pytest.mark.parametrize("seed", range(6))
+def test_gpma_lock_sliding_window(seed):
+    """NEXT-2: GPMA inserts + lazy deletes on configs[0] streams, layout parity every slide."""
+    sw = config_stream(0, seed=200 + seed)
+    V = 1024
+    k0, v0 = sw.initial()
+    g = Gpma.gpma_create(V, k0.to(DEV), v0.to(DEV), algorithm=1)
+    o = O.Oracle(V, k0, v0, algorithm=1)
+    for s in range(4):
+        dk, ik, iv = sw.slide(s)
+        g.delete(dk.to(DEV))
+        g.insert(ik.to(DEV), iv.to(DEV))
+        o.delete(dk)
+        o.insert(ik, iv)
+        assert g.gpma_stats()["last_rounds"] == o.rounds
+        assert_same_layout(g, o, what=f"gpma seed {seed} slide {s}")
+    assert_same_csr(g, o)
+
+
+@pytest.mark.parametrize("seed", range(4))
+def test_gpma_lock_hot_rows_and_doubling(seed):
+    rng = np.random.default_rng(seed)
+    V = 64
+    g = Gpma.gpma_create(V, None, None, algorithm=1)
+    o = O.Oracle(V, [], [], algorithm=1)
+    for step in range(12):
+        b = int(rng.integers(50, 400))
+        ks = _keys(rng.integers(0, 8, b), rng.integers(0, V, b))
+        vs = rng.integers(0, 1 << 31, len(ks)).tolist()
+        g.insert(keys_t(ks), vals_t(vs))
+        o.insert(ks, vs)
+        assert_same_layout(g, o, what=f"gpma hot seed {seed} step {step}")
+    assert g.gpma_stats()["resizes"] == o.stats()["resizes"] > 0
