@@ -341,9 +341,9 @@ def run_gpma(args, rank, world, lrank):
 
 def batch_sweep(dev, batches=(100, 1_000, 10_000, 100_000, 1_000_000)):
     """Update throughput vs batch size (Fig. 7) on configs[1]
-    (Pokec-shaped, 15M-edge window): per B a fresh store from the initial window, 3 warm-up
-    slides, then slides until >= 2M updates (>= 10 slides); slide = DELETE(B oldest) +
-    INSERT(B next), CUDA-event timed."""
+    (Pokec-shaped, 15M-edge window), for GPMA+ (Alg. 4) and GPMA (Alg. 1, lock-based): per B a
+    fresh store from the initial window, 3 warm-up slides, then slides until >= 2M updates
+    (>= 10 slides; GPMA: 5 slides); slide = DELETE(B oldest) + INSERT(B next), CUDA events."""
     from paper_journals_pvldb_shalht17_b200 import Gpma
     cfg = CONFIGS[1]
     sw = config_stream(1, device=dev)
@@ -353,29 +353,37 @@ def batch_sweep(dev, batches=(100, 1_000, 10_000, 100_000, 1_000_000)):
     with torch.cuda.stream(s):
         k0, v0 = sw.initial()
         for B in batches:
-            n_meas = max(10, (2_000_000 + 2 * B - 1) // (2 * B))
-            n_meas = min(n_meas, avail // B - 3)
-            g = Gpma.gpma_create(cfg.V, k0.contiguous(), v0.contiguous(), stream=s)
-            times = []
-            pos = 0
-            for it in range(3 + n_meas):
-                dk = sw.keys[pos:pos + B]
-                ik = sw.keys[sw.window + pos: sw.window + pos + B]
-                iv = sw.vals[sw.window + pos: sw.window + pos + B]
-                pos += B
-                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-                e0.record(s)
-                g.gpma_update_batch(dk, None, 1, stream=s)
-                g.gpma_update_batch(ik, iv, 0, stream=s)
-                e1.record(s)
-                e1.synchronize()
-                if it >= 3:
-                    times.append(e0.elapsed_time(e1))
-            del g
-            t = np.array(times)
-            res.append({"batch": B, "slides": len(times), "updates_per_s": 2 * B / (t.mean() / 1e3),
-                        "ms_per_slide_mean": float(t.mean()), "ms_p50": float(np.percentile(t, 50)),
-                        "ms_p99": float(np.percentile(t, 99))})
+            point = {"batch": B}
+            for alg, name in ((0, "gpma_plus"), (1, "gpma")):
+                n_meas = max(10, (2_000_000 + 2 * B - 1) // (2 * B)) if alg == 0 else 5
+                n_meas = min(n_meas, avail // B - 3)
+                g = Gpma.gpma_create(cfg.V, k0.contiguous(), v0.contiguous(), algorithm=alg, stream=s)
+                times, rounds = [], []
+                pos = 0
+                for it in range(3 + n_meas):
+                    dk = sw.keys[pos:pos + B]
+                    ik = sw.keys[sw.window + pos: sw.window + pos + B]
+                    iv = sw.vals[sw.window + pos: sw.window + pos + B]
+                    pos += B
+                    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                    e0.record(s)
+                    g.gpma_update_batch(dk, None, 1, stream=s)
+                    g.gpma_update_batch(ik, iv, 0, stream=s)
+                    e1.record(s)
+                    e1.synchronize()
+                    if it >= 3:
+                        times.append(e0.elapsed_time(e1))
+                        if alg == 1:
+                            rounds.append(g.gpma_stats()["last_rounds"])
+                del g
+                t = np.array(times)
+                point[name] = {"slides": len(times), "updates_per_s": 2 * B / (t.mean() / 1e3),
+                               "ms_per_slide_mean": float(t.mean()), "ms_p50": float(np.percentile(t, 50)),
+                               "ms_p99": float(np.percentile(t, 99))}
+                if alg == 1:
+                    point[name]["rounds_mean"] = float(np.mean(rounds))
+            point["gpma_plus_speedup"] = point["gpma_plus"]["updates_per_s"] / point["gpma"]["updates_per_s"]
+            res.append(point)
     return {"workload": "configs[1] pokec-shaped (V=1.6M, 15M-edge window)", "points": res}
 
 
