@@ -112,17 +112,15 @@ class Clocks:
 
 # ------------------------------------------------------------------ algorithmic bytes
 def algo_bytes(kernel: str, cap: int, V: int, L: int, nnz: int, dtype_bytes: int = 8) -> int | None:
-    """Algorithmic bytes of ONE launch of the kernel."""
-    if kernel in ("k_pr_push", "k_pr_push_win"):  # key+val of every slot, contrib once per vertex, y RMW once
-        return 12 * cap + dtype_bytes * V + 2 * dtype_bytes * V
-    if kernel == "k_cc_hook":      # read key+val of every slot, parent array read+write once
-        return 12 * cap + 8 * V
-    if kernel == "k_pr_outdeg":
-        return 12 * cap + 4 * V
-    if kernel == "k_exp_leafcount":
-        return 12 * cap + 8 * (cap // L)
-    if kernel == "k_exp_write":    # read slots + leaf bases, write col/val + row_ptr
-        return 12 * cap + 8 * (cap // L) + 8 * nnz + 8 * (V + 1)
+    """Algorithmic bytes of ONE launch, from SURVEY.md §8(d)'s per-unit figures (keys 8 B +
+    values 4 B per slot): PR push 12·cap + 8·V + 8·E per iteration; CC hooking round
+    12·cap + 8·E; export 12·cap + 8·(V+1) + 8·E.  E = live edges."""
+    if kernel in ("k_pr_push", "k_pr_push_win"):    # slots, x/outdeg per row, scatter-add y[dst]
+        return 12 * cap + 8 * V + 8 * nnz
+    if kernel in ("k_cc_hook", "k_cc_sample"):     # one hooking sweep
+        return 12 * cap + 8 * nnz
+    if kernel == "k_exp_write":
+        return 12 * cap + 8 * (V + 1) + 8 * nnz
     return None
 
 
@@ -489,7 +487,7 @@ def run_gpma_dist(args, rank, world, lrank):
     hbm, peak_kind = peaks()
     st = shard.g.gpma_stats()
     cap = st["capacity"]
-    ab = 12 * cap + 8 * (rows[1] - rows[0]) + 16 * V
+    ab = 12 * cap + 8 * (rows[1] - rows[0]) + 8 * st["live_edges"]   # SURVEY §8(d) PR push
     n_l, tot = prof
     avg = tot / n_l if n_l else float("nan")
     ach = ab / (avg / 1e3) / 1e9 if n_l else None
