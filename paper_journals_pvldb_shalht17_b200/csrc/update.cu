@@ -145,16 +145,17 @@ __global__ void k_lazy_delete(const uint64_t *__restrict__ keys, uint64_t n, con
 }
 
 // Fused level 0 of the level loop (Alg. 4 l.7-15 at the leaves, where nearly every update
-// is absorbed): one warp per group of pending updates that share a target leaf.  The warp
-// loads the leaf (lane l = slot l), counts its live entries with a ballot, tests the leaf
-// bound max_0 (insert) / min_0 (strict delete), and on success merges in registers -- the rank
-// of a live entry is its live rank plus the updates below it, the rank of an update its
-// index plus the live entries below it -- and writes the left-packed leaf back (a one-leaf
-// window has a single piece in the R7 split).  Rejected groups stay pending for level 1.
+// is absorbed).  A warp takes the groups of pending updates (one group per target leaf) that
+// start in its 32-item window and hands them to L-lane sub-warps (32/L groups at a time).  A
+// sub-warp loads its leaf (lane l = slot l), counts the live entries with a ballot, tests the
+// leaf bound max_0 (insert) / min_0 (strict delete) and, on success, merges in registers -- a
+// live entry's rank is its live rank plus the updates below it, an update's rank its index
+// plus the live entries below it -- and writes the left-packed leaf back (a one-leaf window
+// is a single piece of the R7 split).  Rejected groups stay pending for level 1.  Control
+// flow is uniform across the warp (everything predicated), so every shuffle is full-mask.
 __global__ void __launch_bounds__(256) k_level0(const uint64_t *__restrict__ pk, const uint32_t *__restrict__ pv,
                                                 const uint32_t *__restrict__ pt, const uint32_t *__restrict__ p_dev,
-                                                uint64_t *key,
-                                                uint32_t *val, uint32_t *__restrict__ cnt,
+                                                uint64_t *key, uint32_t *val, uint32_t *__restrict__ cnt,
                                                 uint32_t *__restrict__ tmask, uint64_t *__restrict__ head,
                                                 uint64_t *__restrict__ row_offset, uint32_t rb, uint32_t L,
                                                 uint32_t bound, int op, uint32_t *__restrict__ keep,
@@ -162,114 +163,115 @@ __global__ void __launch_bounds__(256) k_level0(const uint64_t *__restrict__ pk,
   if (c->err) return;
   const uint64_t p = *p_dev;                         // pending updates (device-side count)
   const int lane = threadIdx.x & 31;
-  const uint32_t lt = (1u << lane) - 1u;
+  const uint32_t nsub = 32 / L, sub = lane / L, sl = lane % L;
+  const uint32_t submask = (L == 32 ? 0xffffffffu : ((1u << L) - 1u) << (sub * L));
+  const uint32_t below_me = (1u << sl) - 1u;
   const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  const bool ins = op == GPMA_INSERT;
   uint32_t accepted = 0;
   for (uint64_t base = ((blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32) * 32; base < p;
        base += nwarps * 32) {
     const uint64_t jl = base + lane;
     const bool first = jl < p && (jl == 0 || pt[jl] != pt[jl - 1]);
-    uint32_t starts = __ballot_sync(0xffffffffu, first);
-    while (starts) {
-      const int sl = __ffs(starts) - 1;
-      starts &= starts - 1;
-      const uint64_t j0 = base + sl;
-      const uint32_t t = pt[j0];
-      // group end: next start in this window, else scan forward
-      uint64_t j1;
-      if (starts) {
-        j1 = base + (__ffs(starts) - 1);
-      } else {
-        j1 = base + 32;
-        while (true) {                                 // warp-cooperative forward scan
-          const uint64_t jj = j1 + lane;
-          const bool other = jj >= p || pt[jj] != t;
-          const uint32_t b = __ballot_sync(0xffffffffu, other);
-          if (b) { j1 += __ffs(b) - 1; break; }
-          j1 += 32;
-        }
-        if (j1 > p) j1 = p;
+    const uint32_t S = __ballot_sync(0xffffffffu, first);
+    if (!S) continue;
+    const uint32_t nstart = __popc(S);
+    // end of the window's last group: warp-cooperative forward scan
+    const uint32_t t_last = pt[base + (31 - __clz(S))];
+    uint64_t last_end = base + 32;
+    while (true) {
+      const uint64_t jj = last_end + lane;
+      const bool other = jj >= p || pt[jj] != t_last;
+      const uint32_t bb = __ballot_sync(0xffffffffu, other);
+      if (bb) { last_end += __ffs(bb) - 1; break; }
+      last_end += 32;
+    }
+    if (last_end > p) last_end = p;
+    for (uint32_t it = 0; it * nsub < nstart; ++it) {
+      const uint32_t gi = it * nsub + sub;
+      const bool have = gi < nstart;
+      uint64_t j0 = 0, j1 = 0;
+      if (have) {
+        j0 = base + __fns(S, 0, gi + 1);
+        j1 = gi + 1 < nstart ? base + __fns(S, 0, gi + 2) : last_end;
       }
+      const uint32_t t = have ? pt[j0] : 0u;
       const uint32_t u = (uint32_t)(j1 - j0);
       const uint64_t lb = (uint64_t)t * L;
       uint64_t ks = KEY_NONE;
       uint32_t vs = 0;
-      if (lane < (int)L) {
-        ks = key[lb + lane];
-        vs = val[lb + lane];
+      if (have) {
+        ks = key[lb + sl];
+        vs = val[lb + sl];
       }
-      const bool live = lane < (int)L && ks != KEY_NONE && vs != VAL_TOMB;
-      const uint32_t lb_live = __ballot_sync(0xffffffffu, live);
-      const uint32_t n = __popc(lb_live);
-      bool ok;
-      if (op == GPMA_INSERT) ok = u <= bound && n + u <= bound;
-      else ok = u <= n && n - u >= bound;
-      if (!ok) {
-        for (uint64_t j = j0 + lane; j < j1; j += 32) keep[j] = 1u;
-        continue;
-      }
+      const bool live = have && ks != KEY_NONE && vs != VAL_TOMB;
+      const uint32_t lbits = (__ballot_sync(0xffffffffu, live) & submask) >> (sub * L);
+      const uint32_t n = __popc(lbits);
+      const bool ok = have && (ins ? (u <= bound && n + u <= bound) : (u <= n && n - u >= bound));
       uint64_t uk = KEY_NONE;
       uint32_t uv = 0;
-      if (lane < (int)u) {
-        uk = pk[j0 + lane];
-        uv = pv[j0 + lane];
+      if (ok && sl < u) {
+        uk = pk[j0 + sl];
+        uv = pv[j0 + sl];
       }
-      // merged ranks
       uint32_t below_u = 0, below_l = 0;
-      for (uint32_t i = 0; i < u; ++i) below_u += __shfl_sync(0xffffffffu, uk, i) < ks;
-      for (uint32_t i = 0; i < L; ++i) {
-        const uint64_t ki = __shfl_sync(0xffffffffu, ks, i);
-        below_l += ((lb_live >> i) & 1u) && ki < uk;
+      bool drop = false;
+      for (uint32_t i = 0; i < L; ++i) {                // merged ranks (width-L shuffles)
+        const uint64_t ui = __shfl_sync(0xffffffffu, uk, i, L);
+        const uint64_t ki = __shfl_sync(0xffffffffu, ks, i, L);
+        below_u += i < u && ui < ks;
+        below_l += ((lbits >> i) & 1u) && ki < uk;
+        drop |= !ins && live && i < u && ui == ks;
       }
-      bool drop = false;                               // (every lane shuffles: full mask)
-      if (op != GPMA_INSERT)
-        for (uint32_t i = 0; i < u; ++i) {
-          const uint64_t ki = __shfl_sync(0xffffffffu, uk, i);   // not short-circuited
-          drop |= live && ki == ks;
+      const uint32_t N = ins ? n + u : n - u;
+      const uint32_t live_rank = __popc(lbits & below_me);
+      const uint32_t lpos = ins ? live_rank + below_u : live_rank - below_u;
+      const uint32_t upos = sl + below_l;
+      // new first key (held by the lane whose entry lands at 0) and the old one
+      const bool l0 = live && !drop && lpos == 0;
+      const bool u0 = ins && ok && sl < u && upos == 0;
+      const uint32_t b0 = ((__ballot_sync(0xffffffffu, l0 || u0) & submask) >> (sub * L));
+      const uint64_t h_new = __shfl_sync(0xffffffffu, l0 ? ks : uk, b0 ? __ffs(b0) - 1 : 0, L);
+      const uint64_t h_old = __shfl_sync(0xffffffffu, ks, 0, L);
+      __syncwarp();
+      if (ok) {
+        if (live && !drop) {
+          key[lb + lpos] = ks;
+          val[lb + lpos] = vs;
+          if (is_guard_key(ks)) row_offset[(ks >> 32) - rb + 1] = lb + lpos;
         }
-      const uint32_t N = op == GPMA_INSERT ? n + u : n - u;
-      const uint32_t live_rank = __popc(lb_live & lt);
-      __syncwarp();
-      // new first key of the leaf (held by the lane whose entry lands at position 0)
-      // (a lane may hold both a live entry and an update: pick the one that lands at 0)
-      const bool l0 = live && !drop && (op == GPMA_INSERT ? live_rank + below_u : live_rank - below_u) == 0;
-      const bool u0 = op == GPMA_INSERT && lane < (int)u && lane + below_l == 0;
-      const uint32_t b0 = __ballot_sync(0xffffffffu, l0 || u0);
-      const uint64_t h_new = N ? __shfl_sync(0xffffffffu, l0 ? ks : uk, b0 ? __ffs(b0) - 1 : 0) : KEY_NONE;
-      const uint64_t h_old = __shfl_sync(0xffffffffu, ks, 0);   // first occupied key before
-      // write entries at their merged position, then clear the tail
-      if (live && !drop) {
-        const uint32_t pos = op == GPMA_INSERT ? live_rank + below_u : live_rank - below_u;
-        key[lb + pos] = ks;
-        val[lb + pos] = vs;
-        if (is_guard_key(ks)) row_offset[(ks >> 32) - rb + 1] = lb + pos;
-      }
-      if (op == GPMA_INSERT && lane < (int)u) {
-        const uint32_t pos = lane + below_l;
-        key[lb + pos] = uk;
-        val[lb + pos] = uv;
+        if (ins && sl < u) {
+          key[lb + upos] = uk;
+          val[lb + upos] = uv;
+        }
       }
       __syncwarp();
-      if (lane < (int)L && lane >= (int)N) {
-        key[lb + lane] = KEY_NONE;
-        val[lb + lane] = 0;
+      if (ok && sl >= N) {
+        key[lb + sl] = KEY_NONE;
+        val[lb + sl] = 0;
       }
-      for (uint64_t j = j0 + lane; j < j1; j += 32) keep[j] = 0u;
-      if (lane == 0) {
+      if (have)
+        for (uint64_t j = j0 + sl; j < j1; j += L) keep[j] = ok ? 0u : 1u;
+      if (ok && sl == 0) {
         cnt[t] = N;
         tmask[t] = 0u;
-        if (h_new != h_old) {
+        if (h_new != h_old && N) {
           head[t] = h_new;
           // empty leaves to the left carry this head (R9): leave them to the final fix-up
-          if (!N || (t > 0 && key[lb - L] == KEY_NONE)) {
+          if (t > 0 && key[lb - L] == KEY_NONE) {
             const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
             dirty[d] = make_uint2(t, 1u);
           }
+        }
+        if (!N) {   // an emptied leaf (strict delete with min_0 = 0): the fix-up recomputes it
+          const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
+          dirty[d] = make_uint2(t, 1u);
         }
         ++accepted;
       }
     }
   }
+  accepted = __reduce_add_sync(0xffffffffu, accepted);
   if (lane == 0 && accepted) atomicAdd((unsigned long long *)&c->windows_rewritten, (unsigned long long)accepted);
 }
 
