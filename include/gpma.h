@@ -22,7 +22,14 @@
  *   - Every function returns a gpma_status.  Argument, range and reserved-value
  *     errors are detected before anything is mutated (no partial batch).  A CUDA
  *     error poisons the handle; later calls return GPMA_ERR_POISONED.
- *   - A handle is not thread-safe; use it from one host thread / stream at a time.
+ *   - Concurrency.  Calls that mutate the store (create, update_batch, destroy) are
+ *     exclusive: nothing else may run on the handle meanwhile.  The read-only analytics
+ *     BFS (gpma_bfs, gpma_bfs_init/level), CC (gpma_cc, gpma_cc_round), PageRank
+ *     (gpma_pagerank*, gpma_pr_push/update), export (gpma_export_csr) and the query buffer
+ *     (gpma_query_*) each own a private scratch + control block, so DIFFERENT analytics
+ *     may run at the same time from different host threads, each on its own stream
+ *     (the caller orders those streams after the last update and before the next one).
+ *     Two calls of the SAME analytic on one handle must not overlap.
  *   - All compute runs in the sm_100a kernels of this library; there is no CPU path.
  */
 #ifndef GPMA_H

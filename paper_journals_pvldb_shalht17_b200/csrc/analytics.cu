@@ -265,24 +265,26 @@ gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
 // shards); the owned rows of the frontier are expanded and newly reached vertices get
 // `depth`.  *frontier = the frontier size (0: the traversal is over, nothing expanded).
 gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontier, cudaStream_t s) {
+  Scratch &X = g->an[AN_BFS];
+  ScanScope scan_scope_(X.scan);
   const uint64_t V = g->V, nl = g->cap / g->L;
-  GP_CHECK(g, ensure(g->b_an[0], (V + 1) * 4, s));
-  GP_CHECK(g, ensure(g->b_an[2], (std::max<uint64_t>(V, nl) + 2) * 8, s));
-  GP_CHECK(g, ensure(g->b_an[3], (V / 32 + 2) * 4, s));
-  GP_CHECK(g, ensure(g->b_misc, (nl + 2) * 4, s));
-  uint32_t *list = (uint32_t *)g->b_an[0].p;
-  uint64_t *off = (uint64_t *)g->b_an[2].p;
-  uint32_t *act = (uint32_t *)g->b_an[2].p;          // shares off's buffer: never both in a level
+  GP_CHECK(g, ensure(X.b[0], (V + 1) * 4, s));
+  GP_CHECK(g, ensure(X.b[2], (std::max<uint64_t>(V, nl) + 2) * 8, s));
+  GP_CHECK(g, ensure(X.b[3], (V / 32 + 2) * 4, s));
+  GP_CHECK(g, ensure(X.misc, (nl + 2) * 4, s));
+  uint32_t *list = (uint32_t *)X.b[0].p;
+  uint64_t *off = (uint64_t *)X.b[2].p;
+  uint32_t *act = (uint32_t *)X.b[2].p;          // shares off's buffer: never both in a level
   uint32_t *apos = act + nl + 1;
-  uint32_t *alist = (uint32_t *)g->b_misc.p;
-  uint32_t *bm = (uint32_t *)g->b_an[3].p;
-  uint32_t *F_d = reinterpret_cast<uint32_t *>(&g->ctrl_d->sum);
+  uint32_t *alist = (uint32_t *)X.misc.p;
+  uint32_t *bm = (uint32_t *)X.b[3].p;
+  uint32_t *F_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum);
   const uint32_t *tmask = tmask_of(g);
   GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
   GP_LAUNCH(g, k_bfs_frontier, grid_for(V), TA, 0, s, levels, (uint32_t)V, depth - 1, bm, F_d);
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
-  const uint32_t F = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
+  const uint32_t F = (uint32_t)(X.ctrl_h->sum & 0xFFFFFFFFu);
   *frontier = F;
   if (!F) return GPMA_OK;
   if (F <= BFS_SPARSE_F) {
@@ -290,13 +292,13 @@ gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontie
     GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, F_d);
     GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, g->rb, g->nr, off);
     scan_u64(g, off, off, F, s);
-    GP_LAUNCH(g, k_bfs_expand, MAX_RESIDENT_BLOCKS, TA, 0, s, list, F, off, g->row_offset, g->key, tmask, g->L,
+    GP_LAUNCH(g, k_bfs_expand, grid_cap(), TA, 0, s, list, F, off, g->row_offset, g->key, tmask, g->L,
               levels, depth, g->rb);
   } else {
     GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, act);
     scan_u32(g, act, apos, nl, s);
     GP_LAUNCH(g, k_bfs_leaf_list, grid_for(nl), TA, 0, s, act, apos, nl, alist);
-    GP_LAUNCH(g, k_bfs_sweep, MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask, g->L, alist, apos + nl, bm, levels,
+    GP_LAUNCH(g, k_bfs_sweep, grid_cap(), TA, 0, s, g->key, tmask, g->L, alist, apos + nl, bm, levels,
               depth);
   }
   GP_CHECK(g, cudaGetLastError());
@@ -447,33 +449,37 @@ __global__ void k_cc_changed(const uint32_t *__restrict__ a, const uint32_t *__r
 // the element-wise minimum of other shards' labels): sampled round, compression, full pass,
 // full compression.  *changed = vertices whose label moved (0 on every shard = fixpoint).
 gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cudaStream_t s) {
+  Scratch &X = g->an[AN_CC];
+  ScanScope scan_scope_(X.scan);
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(g->b_an[1], (V + 1) * 4, s));
-  uint32_t *prev = (uint32_t *)g->b_an[1].p;
+  GP_CHECK(g, ensure(X.b[1], (V + 1) * 4, s));
+  uint32_t *prev = (uint32_t *)X.b[1].p;
   const uint32_t *tmask = tmask_of(g);
   if (init) GP_LAUNCH(g, k_cc_init, grid_for(V), TA, 0, s, labels, g->V);
   GP_CHECK(g, cudaMemcpyAsync(prev, labels, V * 4, cudaMemcpyDeviceToDevice, s));
-  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
+  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
-  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
+  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
-  GP_CHECK(g, cudaMemsetAsync(&g->ctrl_d->sum, 0, 8, s));
-  GP_LAUNCH(g, k_cc_changed, grid_for(V), TA, 0, s, labels, prev, g->V, g->ctrl_d);
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, &g->ctrl_d->sum, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaMemsetAsync(&X.ctrl_d->sum, 0, 8, s));
+  GP_LAUNCH(g, k_cc_changed, grid_for(V), TA, 0, s, labels, prev, g->V, X.ctrl_d);
+  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, &X.ctrl_d->sum, 8, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
-  *changed = g->ctrl_h->sum;
+  *changed = X.ctrl_h->sum;
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
 
 gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s) {
-  GP_CHECK(g, ensure(g->b_an[0], ((uint64_t)g->V + 1) * 4, s));
-  uint32_t *p = (uint32_t *)g->b_an[0].p;
+  Scratch &X = g->an[AN_CC];
+  ScanScope scan_scope_(X.scan);
+  GP_CHECK(g, ensure(X.b[0], ((uint64_t)g->V + 1) * 4, s));
+  uint32_t *p = (uint32_t *)X.b[0].p;
   const uint32_t *tmask = tmask_of(g);
   GP_LAUNCH(g, k_cc_init, grid_for(g->V), TA, 0, s, p, g->V);
-  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->cap, g->L, p);
+  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
   GP_LAUNCH(g, k_cc_compress, grid_for(g->V), TA, 0, s, p, g->V);
-  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4), TA, 0, s, g->key, tmask, g->L, g->cap, p);
+  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
   GP_LAUNCH(g, k_cc_final, grid_for(g->V), TA, 0, s, p, labels, g->V);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
@@ -670,14 +676,16 @@ static uint32_t pr_passes(uint64_t ybytes) {
 template <typename T>
 static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_iter, int *iters,
                               cudaStream_t s) {
+  Scratch &X = g->an[AN_PR];
+  ScanScope scan_scope_(X.scan);
   using A = typename PrAcc<T>::A;
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(g->b_an[1], (V + 1) * sizeof(A), s));
-  GP_CHECK(g, ensure(g->b_an[2], (V + 1) * sizeof(A), s));
-  GP_CHECK(g, ensure(g->b_an[3], 4 * sizeof(double), s));
+  GP_CHECK(g, ensure(X.b[1], (V + 1) * sizeof(A), s));
+  GP_CHECK(g, ensure(X.b[2], (V + 1) * sizeof(A), s));
+  GP_CHECK(g, ensure(X.b[3], 4 * sizeof(double), s));
   const uint32_t *deg = g->deg;
-  A *contrib = (A *)g->b_an[1].p, *y = (A *)g->b_an[2].p;
-  double *acc = (double *)g->b_an[3].p;   // [0],[1] dangling ping-pong, [2] error
+  A *contrib = (A *)X.b[1].p, *y = (A *)X.b[2].p;
+  double *acc = (double *)X.b[3].p;   // [0],[1] dangling ping-pong, [2] error
   const uint32_t passes = pr_passes(V * sizeof(A));
   GP_CHECK(g, cudaMemsetAsync(acc, 0, 4 * sizeof(double), s));
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
@@ -685,7 +693,7 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   while (it < max_iter) {
     // destination passes: random REDs run ~3x faster while their target fits in L2
     for (uint32_t q = 0; q < passes; ++q)
-      GP_LAUNCH(g, (k_pr_push_win<A, 4>), MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
+      GP_LAUNCH(g, (k_pr_push_win<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
                 g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes));
     GP_CHECK(g, cudaMemsetAsync(acc + 2, 0, sizeof(double), s));
     GP_CHECK(g, cudaMemsetAsync(acc + (cur ^ 1), 0, sizeof(double), s));
@@ -693,10 +701,10 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
               acc + (cur ^ 1), acc + 2);
     cur ^= 1;
     ++it;
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, acc + 2, 8, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum2, acc + 2, 8, cudaMemcpyDeviceToHost, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
     double e;
-    memcpy(&e, &g->ctrl_h->sum2, 8);
+    memcpy(&e, &X.ctrl_h->sum2, 8);
     if (e < tol) break;
   }
   if (iters) *iters = it;
@@ -745,14 +753,16 @@ __global__ void k_prd_update(double *__restrict__ x, unsigned long long *__restr
 }
 
 gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
-  GP_CHECK(g, ensure(g->b_an[1], ((uint64_t)g->nr + 1) * 8, s));
-  unsigned long long *contrib = (unsigned long long *)g->b_an[1].p;
+  Scratch &X = g->an[AN_PR];
+  ScanScope scan_scope_(X.scan);
+  GP_CHECK(g, ensure(X.b[1], ((uint64_t)g->nr + 1) * 8, s));
+  unsigned long long *contrib = (unsigned long long *)X.b[1].p;
   unsigned long long *yy = (unsigned long long *)y;
   if (init) GP_LAUNCH(g, k_prd_init, grid_for(g->V), TA, 0, s, x, g->V);
   GP_LAUNCH(g, k_prd_contrib, grid_for(g->nr), TA, 0, s, x, g->deg, g->rb, g->nr, contrib, yy, g->V);
   const uint32_t passes = pr_passes((uint64_t)g->V * 8);
   for (uint32_t q = 0; q < passes; ++q)
-    GP_LAUNCH(g, (k_pr_push_win<unsigned long long, 4>), MAX_RESIDENT_BLOCKS, TA, 0, s, g->key, tmask_of(g),
+    GP_LAUNCH(g, (k_pr_push_win<unsigned long long, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g),
               g->head, g->L, g->cap, contrib, yy, g->rb, g->nr, (uint32_t)((uint64_t)g->V * q / passes),
               (uint32_t)((uint64_t)g->V * (q + 1) / passes));
   GP_CHECK(g, cudaGetLastError());
@@ -760,13 +770,15 @@ gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
 }
 
 gpma_status pr_update(gpma *g, double *x, uint64_t *y, double d, double *err, cudaStream_t s) {
-  double *e_d = reinterpret_cast<double *>(&g->ctrl_d->sum2);
+  Scratch &X = g->an[AN_PR];
+  ScanScope scan_scope_(X.scan);
+  double *e_d = reinterpret_cast<double *>(&X.ctrl_d->sum2);
   GP_CHECK(g, cudaMemsetAsync(e_d, 0, 8, s));
   GP_LAUNCH(g, k_prd_update, grid_for(g->V), TA, 0, s, x, (unsigned long long *)y, g->V, d, e_d);
   GP_CHECK(g, cudaMemsetAsync(y + g->V, 0, 8, s));
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum2, e_d, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum2, e_d, 8, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
-  memcpy(err, &g->ctrl_h->sum2, 8);
+  memcpy(err, &X.ctrl_h->sum2, 8);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
@@ -847,22 +859,24 @@ __global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ k
 
 gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val, uint64_t cap_nnz,
                        uint64_t *nnz_out, cudaStream_t s) {
+  Scratch &X = g->an[AN_EXPORT];
+  ScanScope scan_scope_(X.scan);
   const uint64_t nl = g->cap / g->L;
-  GP_CHECK(g, ensure(g->b_lpre, (nl + 1) * 8, s));
-  uint64_t *lc = (uint64_t *)g->b_lpre.p;
+  GP_CHECK(g, ensure(X.lpre, (nl + 1) * 8, s));
+  uint64_t *lc = (uint64_t *)X.lpre.p;
   GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gcnt_of(g), nl, lc);
   scan_u64(g, lc, lc, nl, s);
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, lc + nl, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, lc + nl, 8, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
-  uint64_t nnz = g->ctrl_h->sum;
+  uint64_t nnz = X.ctrl_h->sum;
   if (nnz_out) *nnz_out = nnz;
   if (!col) return GPMA_OK;
   if (cap_nnz < nnz) {
-    g->err = "export_csr: nnz_capacity too small";
+    set_err(g, "export_csr: nnz_capacity too small");
     return GPMA_ERR_INVALID_ARG;
   }
   GP_CHECK(g, cudaMemsetAsync(row_ptr, 0, 8, s));
-  GP_LAUNCH(g, k_exp_write, grid_for(g->cap / 4), TA, 0, s, g->key, g->val, tmask_of(g), g->L, g->cap, lc,
+  GP_LAUNCH(g, k_exp_write, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, g->val, tmask_of(g), g->L, g->cap, lc,
             row_ptr, col, val, g->rb);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;

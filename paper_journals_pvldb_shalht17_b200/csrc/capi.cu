@@ -58,7 +58,10 @@ struct Out {
 gpma_status begin(gpma *g) {
   if (!g) return GPMA_ERR_INVALID_ARG;
   if (g->poisoned) return GPMA_ERR_POISONED;
-  g->err.clear();
+  {
+    std::lock_guard<std::mutex> lk(g->mu);
+    g->err.clear();
+  }
   return GPMA_OK;
 }
 
@@ -104,6 +107,8 @@ gpma_status apply_config(gpma *g, const gpma_config *cfg, uint32_t *leaf, uint64
   return GPMA_OK;
 }
 
+void free_handle(gpma *g);
+
 gpma *new_handle(uint32_t V) {
   gpma *g = new (std::nothrow) gpma();
   if (!g) return nullptr;
@@ -116,6 +121,15 @@ gpma *new_handle(uint32_t V) {
     return nullptr;
   }
   memset(g->ctrl_h, 0, sizeof(gp::Ctrl));
+  for (gp::Scratch &x : g->an) {
+    if (cudaMalloc((void **)&x.ctrl_d, sizeof(gp::Ctrl)) != cudaSuccess ||
+        cudaMallocHost((void **)&x.ctrl_h, sizeof(gp::Ctrl)) != cudaSuccess) {
+      cudaGetLastError();
+      free_handle(g);
+      return nullptr;
+    }
+    memset(x.ctrl_h, 0, sizeof(gp::Ctrl));
+  }
   return g;
 }
 
@@ -127,9 +141,12 @@ void free_handle(gpma *g) {
                     &g->b_hf, &g->b_widx, &g->b_wfirst, &g->b_acc, &g->b_aidx, &g->b_alist, &g->b_nw,
                     &g->b_woff, &g->b_keep2, &g->b_kpos, &g->b_lpre, &g->b_wk, &g->b_wv, &g->b_dirty,
                     &g->b_scan, &g->b_hist, &g->b_stage[0], &g->b_stage[1], &g->b_stage[2],
-                    &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3,
-                    &g->b_an[0], &g->b_an[1], &g->b_an[2], &g->b_an[3]};
+                    &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3};
   for (DevBuf *b : bufs) gp::release(*b, s);
+  for (gp::Scratch &x : g->an) {
+    DevBuf *xb[] = {&x.b[0], &x.b[1], &x.b[2], &x.b[3], &x.misc, &x.lpre, &x.scan, &x.stage[0], &x.stage[1]};
+    for (DevBuf *b : xb) gp::release(*b, s);
+  }
   if (g->key) cudaFreeAsync(g->key, s);
   if (g->val) cudaFreeAsync(g->val, s);
   if (g->cnt) cudaFreeAsync(g->cnt, s);
@@ -140,6 +157,10 @@ void free_handle(gpma *g) {
   for (cudaEvent_t e : g->ev_pool) cudaEventDestroy(e);
   if (g->ctrl_d) cudaFree(g->ctrl_d);
   if (g->ctrl_h) cudaFreeHost(g->ctrl_h);
+  for (gp::Scratch &x : g->an) {
+    if (x.ctrl_d) cudaFree(x.ctrl_d);
+    if (x.ctrl_h) cudaFreeHost(x.ctrl_h);
+  }
   cudaGetLastError();
   delete g;
 }
@@ -535,7 +556,7 @@ gpma_status gpma_pr_update(gpma_t *g, double *x, uint64_t *y, double damping, do
   return end(g, gp::pr_update(g, x, y, damping, err, (cudaStream_t)stream));
 }
 
-uint64_t gpma_kernel_launches(const gpma_t *g) { return g ? g->launches : 0; }
+uint64_t gpma_kernel_launches(const gpma_t *g) { return g ? g->launches.load() : 0; }
 
 const char *gpma_status_string(gpma_status s) {
   switch (s) {

@@ -45,30 +45,50 @@ static size_t take_event(gpma *g) {
   return g->ev_used++;
 }
 
-bool prof_begin(gpma *g, const char *name, cudaStream_t s) {
+long prof_begin(gpma *g, const char *name, cudaStream_t s) {
   while (*name == '(') ++name;            // GP_LAUNCH((k<T, U>), ...) stringises the parentheses
   if (g->prof_filter != "*") {
     // exact match on the kernel name without template arguments
     const char *lt = strchr(name, '<');
     size_t n = lt ? (size_t)(lt - name) : strlen(name);
-    if (g->prof_filter.size() != n || strncmp(g->prof_filter.c_str(), name, n) != 0) return false;
+    if (g->prof_filter.size() != n || strncmp(g->prof_filter.c_str(), name, n) != 0) return -1;
   }
+  std::lock_guard<std::mutex> lk(g->mu);
   size_t e0 = take_event(g), e1 = take_event(g);
   cudaEventRecord(g->ev_pool[e0], s);
   g->prof_recs.push_back({name, e0, e1});
-  return true;
+  return (long)g->prof_recs.size() - 1;
 }
 
-void prof_end(gpma *g, cudaStream_t s) { cudaEventRecord(g->ev_pool[g->prof_recs.back().e1], s); }
+void prof_end(gpma *g, long rec, cudaStream_t s) {
+  std::lock_guard<std::mutex> lk(g->mu);
+  cudaEventRecord(g->ev_pool[g->prof_recs[rec].e1], s);
+}
+
+thread_local DevBuf *tl_scan = nullptr;
+
+int grid_cap() {
+  static const int v = [] {
+    const char *e = getenv("GPMA_GRID_CAP");
+    int c = e ? atoi(e) : 0;
+    return c > 0 ? c : MAX_RESIDENT_BLOCKS;
+  }();
+  return v;
+}
+
+void set_err(gpma *g, const std::string &msg) {
+  std::lock_guard<std::mutex> lk(g->mu);
+  g->err = msg;
+}
 
 gpma_status cuda_fail(gpma *g, cudaError_t e, const char *where) {
   if (e == cudaErrorMemoryAllocation) {
     cudaGetLastError();
-    g->err = std::string("out of device memory in ") + where;
+    set_err(g, std::string("out of device memory in ") + where);
     return GPMA_ERR_OOM;
   }
   g->poisoned = true;
-  g->err = std::string(cudaGetErrorString(e)) + " in " + where;
+  set_err(g, std::string(cudaGetErrorString(e)) + " in " + where);
   return GPMA_ERR_CUDA;
 }
 
@@ -212,8 +232,9 @@ static void scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) 
     GP_LAUNCH(g, k_scan_lookback<T>, 1, SC_THREADS, 0, s, in, out, n, (unsigned long long *)nullptr);
     return;
   }
-  ensure(g->b_scan, (nt + 1) * sizeof(unsigned long long), s);
-  unsigned long long *status = (unsigned long long *)g->b_scan.p;
+  DevBuf &sb = tl_scan ? *tl_scan : g->b_scan;
+  ensure(sb, (nt + 1) * sizeof(unsigned long long), s);
+  unsigned long long *status = (unsigned long long *)sb.p;
   cudaMemsetAsync(status, 0, (nt + 1) * sizeof(unsigned long long), s);
   GP_LAUNCH(g, k_scan_lookback<T>, (unsigned)nt, SC_THREADS, 0, s, in, out, n, status);
 }

@@ -152,9 +152,11 @@ __global__ void k_msbfs_answer(const uint32_t *__restrict__ dst, uint32_t nq, co
 }
 
 gpma_status query_edges(gpma *g, const uint64_t *keys, uint64_t n, uint32_t *vals, uint8_t *found, cudaStream_t s) {
+  Scratch &X = g->an[AN_QUERY];
+  ScanScope scan_scope_(X.scan);
   if (!n) return GPMA_OK;
-  GP_CHECK(g, ensure(g->b_stage[2], n * 8, s));
-  uint64_t *q = (uint64_t *)g->b_stage[2].p;
+  GP_CHECK(g, ensure(X.stage[0], n * 8, s));
+  uint64_t *q = (uint64_t *)X.stage[0].p;
   GP_CHECK(g, cudaMemcpyAsync(q, keys, n * 8, cudaMemcpyDefault, s));
   GP_LAUNCH(g, k_query_edges, grid_for(n), TQ, 0, s, q, n, g->key, g->val, g->head, (uint32_t)(g->cap / g->L),
             g->L, vals, found);
@@ -164,20 +166,22 @@ gpma_status query_edges(gpma *g, const uint64_t *keys, uint64_t n, uint32_t *val
 
 gpma_status query_neighbors(gpma *g, const uint32_t *verts, uint64_t n, uint64_t *row_ptr, uint32_t *col,
                             uint32_t *val, uint64_t cap_nnz, uint64_t *nnz_out, cudaStream_t s) {
-  GP_CHECK(g, ensure(g->b_stage[3], (n + 1) * 4, s));
-  GP_CHECK(g, ensure(g->b_lpre, (n + 1) * 8, s));
-  uint32_t *vq = (uint32_t *)g->b_stage[3].p;
-  uint64_t *rp = (uint64_t *)g->b_lpre.p;
+  Scratch &X = g->an[AN_QUERY];
+  ScanScope scan_scope_(X.scan);
+  GP_CHECK(g, ensure(X.stage[1], (n + 1) * 4, s));
+  GP_CHECK(g, ensure(X.lpre, (n + 1) * 8, s));
+  uint32_t *vq = (uint32_t *)X.stage[1].p;
+  uint64_t *rp = (uint64_t *)X.lpre.p;
   if (n) GP_CHECK(g, cudaMemcpyAsync(vq, verts, n * 4, cudaMemcpyDefault, s));
   if (n) GP_LAUNCH(g, k_query_rowsizes, grid_for(n), TQ, 0, s, vq, n, g->deg, g->rb, g->nr, rp);
   scan_u64(g, rp, rp, n, s);
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, rp + n, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, rp + n, 8, cudaMemcpyDeviceToHost, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
-  const uint64_t nnz = n ? g->ctrl_h->sum : 0;
+  const uint64_t nnz = n ? X.ctrl_h->sum : 0;
   if (nnz_out) *nnz_out = nnz;
   if (!col) return GPMA_OK;
   if (cap_nnz < nnz) {
-    g->err = "query_neighbors: nnz_capacity too small";
+    set_err(g, "query_neighbors: nnz_capacity too small");
     return GPMA_ERR_INVALID_ARG;
   }
   if (row_ptr) GP_CHECK(g, cudaMemcpyAsync(row_ptr, rp, (n + 1) * 8, cudaMemcpyDeviceToDevice, s));
@@ -190,14 +194,16 @@ gpma_status query_neighbors(gpma *g, const uint32_t *verts, uint64_t n, uint64_t
 
 gpma_status query_reachable(gpma *g, const uint32_t *src, const uint32_t *dst, uint64_t n, uint8_t *out,
                             cudaStream_t s) {
+  Scratch &X = g->an[AN_QUERY];
+  ScanScope scan_scope_(X.scan);
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(g->b_an[0], V * 8, s));
-  GP_CHECK(g, ensure(g->b_an[1], V * 8, s));
-  GP_CHECK(g, ensure(g->b_an[2], V * 8, s));
-  GP_CHECK(g, ensure(g->b_stage[3], 2 * 64 * 4 + 16, s));
-  unsigned long long *seen = (unsigned long long *)g->b_an[0].p, *front = (unsigned long long *)g->b_an[1].p,
-                     *next = (unsigned long long *)g->b_an[2].p;
-  uint32_t *qs = (uint32_t *)g->b_stage[3].p, *qd = qs + 64;
+  GP_CHECK(g, ensure(X.b[0], V * 8, s));
+  GP_CHECK(g, ensure(X.b[1], V * 8, s));
+  GP_CHECK(g, ensure(X.b[2], V * 8, s));
+  GP_CHECK(g, ensure(X.stage[1], 2 * 64 * 4 + 16, s));
+  unsigned long long *seen = (unsigned long long *)X.b[0].p, *front = (unsigned long long *)X.b[1].p,
+                     *next = (unsigned long long *)X.b[2].p;
+  uint32_t *qs = (uint32_t *)X.stage[1].p, *qd = qs + 64;
   unsigned long long *flags = (unsigned long long *)(qd + 64);   // [0] alive, [1] resolved
   for (uint64_t b0 = 0; b0 < n; b0 += 64) {
     const uint32_t nq = (uint32_t)std::min<uint64_t>(64, n - b0);

@@ -10,11 +10,14 @@ from __future__ import annotations
 
 import torch
 
+from .fanout import AnalyticsFanout
+
 
 class SlidingWindowPipeline:
     def __init__(self, g, V: int, max_batch: int, nnz_capacity: int, device, rows: int | None = None,
-                 pr_tol: float = 1e-3):
+                 pr_tol: float = 1e-3, concurrent: bool = False):
         self.g, self.V, self.dev, self.pr_tol = g, V, torch.device(device), pr_tol
+        self.fan = AnalyticsFanout(self.dev, priorities=[0, -1, -2, 0]) if concurrent else None
         self.cs = torch.cuda.Stream(self.dev)      # compute
         self.xs = torch.cuda.Stream(self.dev)      # copies
         nr = V if rows is None else rows
@@ -61,11 +64,20 @@ class SlidingWindowPipeline:
         with torch.cuda.stream(s):
             g.gpma_update_batch(kd[:nd], None, 1, stream=s)
             g.gpma_update_batch(ki[:ni], vi[:ni], 0, stream=s)
-            g.gpma_bfs(root, lv, stream=s)
-            g.gpma_cc(lab, stream=s)
-            self.pr_iters.append(g.gpma_pagerank(self.x, warm_start=True, tol_l1=self.pr_tol, stream=s))
-            self.d_x[slot].copy_(self.x, non_blocking=True)
-            self.nnz[slot] = g.gpma_export_csr(rp, col, cv, stream=s)
+            dx = self.d_x[slot]
+
+            def pr(st):
+                it = g.gpma_pagerank(self.x, warm_start=True, tol_l1=self.pr_tol, stream=st)
+                dx.copy_(self.x, non_blocking=True)
+                return it
+            jobs = [pr, lambda st: g.gpma_cc(lab, stream=st), lambda st: g.gpma_bfs(root, lv, stream=st),
+                    lambda st: g.gpma_export_csr(rp, col, cv, stream=st)]
+            if self.fan is not None:          # the read-only analytics side by side (fanout.py)
+                r = self.fan.run(s, jobs)
+            else:
+                r = [j(s) for j in jobs]
+            self.pr_iters.append(r[0])
+            self.nnz[slot] = r[3]
             self.ev_done[slot].record(s)
         self.xs.wait_event(self.ev_done[slot])
         h = self.h_out[slot]
@@ -88,3 +100,7 @@ class SlidingWindowPipeline:
 
     def drain(self):
         torch.cuda.synchronize(self.dev)
+
+    def close(self):
+        if self.fan is not None:
+            self.fan.close()

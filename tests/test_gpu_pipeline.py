@@ -11,7 +11,8 @@ from tests.gpu_helpers import DEV
 pytestmark = pytest.mark.gpu
 
 
-def test_pipeline_matches_oracle():
+@pytest.mark.parametrize("concurrent", [False, True])
+def test_pipeline_matches_oracle(concurrent):
     from paper_journals_pvldb_shalht17_b200 import Gpma
     from paper_journals_pvldb_shalht17_b200.pipeline import SlidingWindowPipeline
     seed = 8
@@ -20,7 +21,7 @@ def test_pipeline_matches_oracle():
     k0, v0 = sw.initial()
     g = Gpma.gpma_create(V, k0.to(DEV), v0.to(DEV))
     o = O.Oracle(V, k0, v0)
-    pipe = SlidingWindowPipeline(g, V, sw.batch, sw.window + sw.batch, DEV, pr_tol=0.0)
+    pipe = SlidingWindowPipeline(g, V, sw.batch, sw.window + sw.batch, DEV, pr_tol=0.0, concurrent=concurrent)
     xo, _ = o.pagerank(tol=0.0, max_iter=100)
     batches = [tuple(t.contiguous().pin_memory() for t in sw.slide(s)) for s in range(4)]
     pipe.stage(0, *batches[0])
@@ -41,3 +42,4 @@ def test_pipeline_matches_oracle():
         xo, _ = o.pagerank(x=xo, tol=0.0, max_iter=100)
         assert np.abs(x.numpy() - xo).max() <= 1e-6
     pipe.drain()
+    pipe.close()
