@@ -47,6 +47,12 @@ __device__ __forceinline__ void load4(const uint64_t *__restrict__ key, const ui
   o.tb = (__ldg(tmask + s4 / L) >> (uint32_t)(s4 % L)) & 0xFu;
 }
 
+__device__ __forceinline__ uint64_t l2_evict_last_policy() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
+
 __device__ __forceinline__ bool live_key(uint64_t k) { return k != KEY_NONE && (uint32_t)k != COL_GUARD; }
 __device__ __forceinline__ bool edge4(const Slot4 &o, int j) { return live_key(o.k[j]) && !((o.tb >> j) & 1u); }
 
@@ -316,14 +322,36 @@ gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
 }
 
 // ------------------------------------------------------------------ CC
-__device__ __forceinline__ uint32_t cc_find(uint32_t *p, uint32_t x) {
+// Parent-array accesses may carry an L2 evict_last hint (H): the 64 MB forest stays resident
+// while the key stream passes through L2 evict-first.
+
+template <bool H>
+__device__ __forceinline__ uint32_t cc_ld(const uint32_t *a, uint64_t pol) {
+  uint32_t v;
+  if (H) asm volatile("ld.relaxed.gpu.global.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(v) : "l"(a), "l"(pol) : "memory");
+  else v = *(const volatile uint32_t *)a;
+  return v;
+}
+
+template <bool H>
+__device__ __forceinline__ void cc_st(uint32_t *a, uint32_t v, uint64_t pol) {
+  if (H) asm volatile("st.relaxed.gpu.global.L2::cache_hint.u32 [%0], %1, %2;" ::"l"(a), "r"(v), "l"(pol) : "memory");
+  else *(volatile uint32_t *)a = v;
+}
+
+template <bool H>
+__device__ __forceinline__ uint32_t cc_cas(uint32_t *a, uint32_t cmp, uint32_t v, uint64_t) {
+  return atomicCAS(a, cmp, v);                 // (atom.cas takes no L2 cache hint on sm_100a)
+}
+
+template <bool H>
+__device__ __forceinline__ uint32_t cc_find(uint32_t *p, uint32_t x, uint64_t pol) {
   // path halving on a forest with parent[x] <= x (roots are the minima)
-  volatile uint32_t *vp = p;
-  uint32_t cur = vp[x];
+  uint32_t cur = cc_ld<H>(p + x, pol);
   if (cur != x) {
     uint32_t prev = x, next;
-    while (cur > (next = vp[cur])) {
-      vp[prev] = next;
+    while (cur > (next = cc_ld<H>(p + cur, pol))) {
+      cc_st<H>(p + prev, next, pol);
       prev = cur;
       cur = next;
     }
@@ -331,17 +359,18 @@ __device__ __forceinline__ uint32_t cc_find(uint32_t *p, uint32_t x) {
   return cur;
 }
 
-__device__ __forceinline__ void cc_hook(uint32_t *p, uint32_t u, uint32_t v) {
-  uint32_t ru = cc_find(p, u), rv = cc_find(p, v);
+template <bool H>
+__device__ __forceinline__ void cc_hook(uint32_t *p, uint32_t u, uint32_t v, uint64_t pol) {
+  uint32_t ru = cc_find<H>(p, u, pol), rv = cc_find<H>(p, v, pol);
   bool repeat;
   do {
     repeat = false;
     if (ru != rv) {
       uint32_t ret;
       if (ru < rv) {
-        if ((ret = atomicCAS(&p[rv], rv, ru)) != rv) { rv = ret; repeat = true; }
+        if ((ret = cc_cas<H>(&p[rv], rv, ru, pol)) != rv) { rv = ret; repeat = true; }
       } else {
-        if ((ret = atomicCAS(&p[ru], ru, rv)) != ru) { ru = ret; repeat = true; }
+        if ((ret = cc_cas<H>(&p[ru], ru, rv, pol)) != ru) { ru = ret; repeat = true; }
       }
     }
   } while (repeat);
@@ -357,10 +386,12 @@ __global__ void k_cc_init(uint32_t *p, uint32_t V) {
 // two edges of every row (Afforest-style neighbour sampling; any edge subset is a valid first
 // round), skipping pairs that already share a parent.  (A CAS-free atomicMin linking of the
 // same sample was measured: it halves this round but leaves 4x more work to the full pass.)
+template <bool H>
 __global__ void __launch_bounds__(TA) k_cc_sample(const uint64_t *__restrict__ key,
                                                   const uint32_t *__restrict__ tmask, uint64_t cap, uint32_t L,
                                                   uint32_t *p) {
   const int lane = threadIdx.x & 31;
+  const uint64_t pol = H ? l2_evict_last_policy() : 0;
   const uint64_t n4 = cap / 4, n4r = (n4 + 31) & ~31ull;
   for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4r;
        t += (uint64_t)gridDim.x * blockDim.x) {
@@ -379,7 +410,7 @@ __global__ void __launch_bounds__(TA) k_cc_sample(const uint64_t *__restrict__ k
       const bool first = (s % L == 0) || pk == KEY_NONE || (pk >> 32) != (sl.k[j] >> 32);
       if (!first) continue;
       uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
-      if (u != v && __ldcg(p + u) != __ldcg(p + v)) cc_hook(p, u, v);
+      if (u != v && cc_ld<H>(p + u, pol) != cc_ld<H>(p + v, pol)) cc_hook<H>(p, u, v, pol);
     }
   }
 }
@@ -394,36 +425,44 @@ __global__ void k_cc_compress(uint32_t *p, uint32_t V) {
   }
 }
 
-__device__ __forceinline__ void cc_group(const Slot4 &sl, uint32_t *p) {
+template <bool H>
+__device__ __forceinline__ void cc_group(const Slot4 &sl, uint32_t *p, uint64_t pol) {
   uint32_t pu[4], pv[4];
 #pragma unroll
   for (int j = 0; j < 4; ++j) {             // independent parent loads first
     pu[j] = pv[j] = 0;
     if (edge4(sl, j)) {
-      pu[j] = __ldcg(p + (uint32_t)(sl.k[j] >> 32));
-      pv[j] = __ldcg(p + (uint32_t)sl.k[j]);
+      pu[j] = cc_ld<H>(p + (uint32_t)(sl.k[j] >> 32), pol);
+      pv[j] = cc_ld<H>(p + (uint32_t)sl.k[j], pol);
     }
   }
 #pragma unroll
   for (int j = 0; j < 4; ++j) {
     if (!edge4(sl, j) || pu[j] == pv[j]) continue;   // same tree already (fast path)
     uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
-    if (u != v) cc_hook(p, u, v);
+    if (u != v) cc_hook<H>(p, u, v, pol);
   }
 }
 
+template <bool H>
 __global__ void __launch_bounds__(TA) k_cc_hook(const uint64_t *__restrict__ key,
                                                 const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
                                                 uint32_t *p) {
+  const uint64_t pol = H ? l2_evict_last_policy() : 0;
   const uint64_t n4 = cap / 4, stride = (uint64_t)gridDim.x * blockDim.x;
   for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4; t += 2 * stride) {
     Slot4 a, b;
     const bool hb = t + stride < n4;
     load4(key, tmask, L, t * 4, a);
     if (hb) load4(key, tmask, L, (t + stride) * 4, b);
-    cc_group(a, p);
-    if (hb) cc_group(b, p);
+    cc_group<H>(a, p, pol);
+    if (hb) cc_group<H>(b, p, pol);
   }
+}
+
+static int cc_hint() {
+  static const int v = [] { const char *e = getenv("GPMA_CC_HINT"); return e ? atoi(e) : 1; }();
+  return v;
 }
 
 __global__ void k_cc_final(uint32_t *p, uint32_t *labels, uint32_t V) {
@@ -457,9 +496,11 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
   const uint32_t *tmask = tmask_of(g);
   if (init) GP_LAUNCH(g, k_cc_init, grid_for(V), TA, 0, s, labels, g->V);
   GP_CHECK(g, cudaMemcpyAsync(prev, labels, V * 4, cudaMemcpyDeviceToDevice, s));
-  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
+  if (cc_hint()) GP_LAUNCH(g, k_cc_sample<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
+  else GP_LAUNCH(g, k_cc_sample<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
-  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
+  if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
+  else GP_LAUNCH(g, k_cc_hook<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
   GP_CHECK(g, cudaMemsetAsync(&X.ctrl_d->sum, 0, 8, s));
   GP_LAUNCH(g, k_cc_changed, grid_for(V), TA, 0, s, labels, prev, g->V, X.ctrl_d);
@@ -477,9 +518,11 @@ gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s) {
   uint32_t *p = (uint32_t *)X.b[0].p;
   const uint32_t *tmask = tmask_of(g);
   GP_LAUNCH(g, k_cc_init, grid_for(g->V), TA, 0, s, p, g->V);
-  GP_LAUNCH(g, k_cc_sample, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
+  if (cc_hint()) GP_LAUNCH(g, k_cc_sample<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
+  else GP_LAUNCH(g, k_cc_sample<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
   GP_LAUNCH(g, k_cc_compress, grid_for(g->V), TA, 0, s, p, g->V);
-  GP_LAUNCH(g, k_cc_hook, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
+  if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
+  else GP_LAUNCH(g, k_cc_hook<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
   GP_LAUNCH(g, k_cc_final, grid_for(g->V), TA, 0, s, p, labels, g->V);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
@@ -575,6 +618,15 @@ __global__ void __launch_bounds__(TA) k_pr_push(const uint64_t *__restrict__ key
   }
 }
 
+// RED with an L2 eviction-priority hint (evict_last keeps the scattered y lines resident
+// while the key stream, loaded evict-first, passes through L2).
+__device__ __forceinline__ void red_add_hint(unsigned long long *p, unsigned long long v, uint64_t pol) {
+  asm volatile("red.global.add.L2::cache_hint.u64 [%0], %1, %2;" ::"l"(p), "l"(v), "l"(pol) : "memory");
+}
+__device__ __forceinline__ void red_add_hint(float *p, float v, uint64_t pol) {
+  asm volatile("red.global.add.L2::cache_hint.f32 [%0], %1, %2;" ::"l"(p), "f"(v), "l"(pol) : "memory");
+}
+
 // Row-window push: warp w sweeps the contiguous slot chunk [beg, end) (leaf aligned).  Keys
 // are sorted, so the sources met along the chunk never decrease: lane j keeps contrib[ub + j]
 // of a 32-row window in a register and every slot fetches its source's contribution with a
@@ -586,8 +638,11 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
                                                     const uint32_t *__restrict__ tmask,
                                                     const uint64_t *__restrict__ head, uint32_t L, uint64_t cap,
                                                     const A *__restrict__ contrib, A *y, uint32_t rb,
-                                                    uint32_t nr, uint32_t dlo, uint32_t dhi) {
+                                                    uint32_t nr, uint32_t dlo, uint32_t dhi, int hint) {
   const int lane = threadIdx.x & 31;
+  uint64_t pol = 0;
+  if (hint == 1) asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
+  if (hint == 2) asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 0.5;" : "=l"(pol));
   const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
   const uint64_t w = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32;
   const uint64_t chunk = (((cap + nwarps - 1) / nwarps) + 32 * U - 1) / (32 * U) * (32 * U);
@@ -621,7 +676,10 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
         const uint32_t off = mine ? u - ub : 0u;
         const bool in = mine && off < 32u;
         const A c = __shfl_sync(0xffffffffu, win, off & 31u);
-        if (in) atomicAdd(&y[dv], c);
+        if (in) {
+          if (hint) red_add_hint(&y[dv], c, pol);
+          else atomicAdd(&y[dv], c);
+        }
         pending &= ~__ballot_sync(0xffffffffu, in);
         if (pending) {                                   // slide the window to the next source
           ub = __reduce_min_sync(0xffffffffu, ((pending >> lane) & 1u) ? u : 0xFFFFFFFFu);
@@ -666,6 +724,13 @@ __global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ 
 // Destination passes of the push (GPMA_PR_PASSES, default 1).  Random REDs run ~3x faster
 // while their target fits in L2 (tools/micro/red_bench.cu), but each pass re-sweeps the keys;
 // at V = 2^24 one pass measured fastest.
+// y REDs carry an L2 evict_last hint (GPMA_PR_HINT=0 disables): push 4.72 -> 3.99 ms / 3 iters
+// at configs[2]
+static int pr_hint() {
+  static const int v = [] { const char *e = getenv("GPMA_PR_HINT"); return e ? atoi(e) : 1; }();
+  return v;
+}
+
 static uint32_t pr_passes(uint64_t ybytes) {
   (void)ybytes;
   uint64_t p = 1;
@@ -694,7 +759,8 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
     // destination passes: random REDs run ~3x faster while their target fits in L2
     for (uint32_t q = 0; q < passes; ++q)
       GP_LAUNCH(g, (k_pr_push_win<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
-                g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes));
+                g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes),
+                pr_hint());
     GP_CHECK(g, cudaMemsetAsync(acc + 2, 0, sizeof(double), s));
     GP_CHECK(g, cudaMemsetAsync(acc + (cur ^ 1), 0, sizeof(double), s));
     GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
@@ -764,7 +830,7 @@ gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
   for (uint32_t q = 0; q < passes; ++q)
     GP_LAUNCH(g, (k_pr_push_win<unsigned long long, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g),
               g->head, g->L, g->cap, contrib, yy, g->rb, g->nr, (uint32_t)((uint64_t)g->V * q / passes),
-              (uint32_t)((uint64_t)g->V * (q + 1) / passes));
+              (uint32_t)((uint64_t)g->V * (q + 1) / passes), pr_hint());
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }

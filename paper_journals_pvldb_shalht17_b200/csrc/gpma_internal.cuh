@@ -74,6 +74,7 @@ struct gpma {
   uint32_t V = 0, L = 0, h = 0, mode = 0;
   uint32_t rb = 0, nr = 0;        // owned rows [rb, rb + nr) (shard, R24); nr = V unsharded
   uint32_t algorithm = 0;         // 0 = GPMA+ (Alg. 4), 1 = GPMA lock-based (Alg. 1)
+  bool rows_indexed = false;      // every owned row has its guard: row_offset locates leaves
   uint64_t cap = 0;
   uint32_t rho0 = 800, rhoh = 4000, tau0 = 9200, tauh = 8000, init_bp = 6000;
   std::vector<uint64_t> tmin, tmax;

@@ -35,6 +35,27 @@ __device__ __forceinline__ uint32_t locate_leaf(const uint64_t *__restrict__ hea
   return lo ? lo - 1 : 0;
 }
 
+// The same leaf through the row index (R8): key (u, v) lies between guard u-1 (slot
+// row_offset[u], leaf a) and guard u (slot row_offset[u+1], leaf b), and head[a] <= guard u-1
+// < key < head[b+1], so the upper bound over head[a..b] equals the global one (row 0: a = 0).
+// A few dependent loads instead of log2(nleaves).  ro == nullptr (raw layouts without
+// guards): the global search.
+__device__ __forceinline__ uint32_t locate_leaf_rows(const uint64_t *__restrict__ head, uint32_t nleaves,
+                                                     const uint64_t *__restrict__ ro, uint32_t rb, uint32_t L,
+                                                     uint64_t k) {
+  if (!ro) return locate_leaf(head, nleaves, k);
+  const uint32_t u = (uint32_t)(k >> 32) - rb;
+  const ulonglong2 r = make_ulonglong2(__ldg(ro + u), __ldg(ro + u + 1));
+  const uint32_t a = (uint32_t)(r.x / L);
+  uint32_t lo = a, hi = min((uint32_t)(r.y / L) + 1, nleaves);
+  while (lo < hi) {
+    uint32_t mid = (lo + hi) >> 1;
+    if (__ldg(head + mid) <= k) lo = mid + 1;
+    else hi = mid;
+  }
+  return lo > a ? lo - 1 : a;
+}
+
 // ------------------------------------------------------------------ validate
 __global__ void k_validate(const uint64_t *__restrict__ keys, const uint32_t *__restrict__ vals,
                            uint64_t n, uint32_t V, uint32_t rb, uint32_t nr, int check_vals, Ctrl *c) {
@@ -58,7 +79,8 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
                           uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
                           uint32_t nleaves, uint32_t L, int op, int mode,
                           uint32_t *__restrict__ keep, uint32_t *__restrict__ tgt, Ctrl *c,
-                          uint32_t *__restrict__ tmask, uint32_t *__restrict__ deg, uint32_t rb) {
+                          uint32_t *__restrict__ tmask, uint32_t *__restrict__ deg, uint32_t rb,
+                          const uint64_t *__restrict__ ro) {
   if (c->err) return;                                // rejected batch: nothing may change
   uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
   uint32_t uniq = 0;
@@ -67,7 +89,7 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
     uint32_t kp = 0, t = 0;
     if (i + 1 == n || sk[i + 1] != k) {
       uniq = 1;
-      t = locate_leaf(head, nleaves, k);
+      t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
       uint64_t base = (uint64_t)t * L, hit = KEY_NONE;
       for (uint32_t p = 0; p < L; ++p) {
         uint64_t x = key[base + p];
@@ -116,12 +138,13 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
 __global__ void k_lazy_delete(const uint64_t *__restrict__ keys, uint64_t n, const uint64_t *__restrict__ key,
                               uint32_t *val, uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
                               uint32_t nleaves, uint32_t L, uint32_t *__restrict__ tmask,
-                              uint32_t *__restrict__ deg, uint32_t rb, const Ctrl *c) {
+                              uint32_t *__restrict__ deg, uint32_t rb, const Ctrl *c,
+                              const uint64_t *__restrict__ ro) {
   if (c->err) return;                                // rejected batch: nothing may change
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
        i += (uint64_t)gridDim.x * blockDim.x) {
     const uint64_t k = keys[i];
-    const uint32_t t = locate_leaf(head, nleaves, k);
+    const uint32_t t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
     const uint64_t base = (uint64_t)t * L;
     for (uint32_t p = 0; p < L; ++p) {
       const uint64_t x = key[base + p];
@@ -885,8 +908,6 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
   uint32_t *wv = (uint32_t *)g->b_wv.p;
   if (m) {
     // positions: edge with unique rank j (pos) and source u goes to j + u
-    int which_unused = 0;
-    (void)which_unused;
     uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p;
     // recompute from the dense list: keep = 1, pos = j
     // (the dense list ek is sorted & unique; place directly)
@@ -896,6 +917,7 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
   }
   GP_LAUNCH(g, k_place_guards, grid_for(g->nr), TB, 0, s, g->rb, g->nr, ek, m, wk, wv);
   GP_CHECK(g, cudaGetLastError());
+  g->rows_indexed = true;      // one guard per owned row from here on (R1)
   return build_from_sorted(g, wk, wv, E, s);
 }
 
@@ -1300,7 +1322,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   const uint64_t nl = g->cap / g->L;
   if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
     GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
-              tmask_of(g), g->deg, g->rb, g->ctrl_d);
+              tmask_of(g), g->deg, g->rb, g->ctrl_d, g->rows_indexed ? g->row_offset : nullptr);
     if ((st = read_ctrl(g, s))) return st;
     g->last.last_unique = n;   // not deduplicated: lazy deletes are idempotent
     return status_of(g);
@@ -1316,7 +1338,8 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   if ((st = level_buffers(g, n, s))) return st;
   uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p, *tgt = (uint32_t *)g->b_tgt.p;
   GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt, g->head,
-            (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb);
+            (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb,
+            g->rows_indexed ? g->row_offset : nullptr);
   scan_u32(g, keep, pos, n, s);
   GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, tgt, (uint64_t *)g->b_pk[0].p,
             (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p, g->ctrl_d);

@@ -15,8 +15,9 @@ from .fanout import AnalyticsFanout
 
 class SlidingWindowPipeline:
     def __init__(self, g, V: int, max_batch: int, nnz_capacity: int, device, rows: int | None = None,
-                 pr_tol: float = 1e-3, concurrent: bool = False):
+                 pr_tol: float = 1e-3, concurrent: bool = False, copy_csr: bool = True):
         self.g, self.V, self.dev, self.pr_tol = g, V, torch.device(device), pr_tol
+        self.copy_csr = copy_csr              # False: the exported CSR stays in HBM (device users)
         self.fan = AnalyticsFanout(self.dev, priorities=[0, -1, -2, 0]) if concurrent else None
         self.cs = torch.cuda.Stream(self.dev)      # compute
         self.xs = torch.cuda.Stream(self.dev)      # copies
@@ -85,9 +86,10 @@ class SlidingWindowPipeline:
         with torch.cuda.stream(self.xs):
             h[0].copy_(lv, non_blocking=True)
             h[1].copy_(lab, non_blocking=True)
-            h[2].copy_(rp, non_blocking=True)
-            h[3][:n].copy_(col[:n], non_blocking=True)
-            h[4][:n].copy_(cv[:n], non_blocking=True)
+            if self.copy_csr:
+                h[2].copy_(rp, non_blocking=True)
+                h[3][:n].copy_(col[:n], non_blocking=True)
+                h[4][:n].copy_(cv[:n], non_blocking=True)
             h[5].copy_(self.d_x[slot], non_blocking=True)
             self.ev_out[slot].record(self.xs)
 
