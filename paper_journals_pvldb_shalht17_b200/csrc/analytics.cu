@@ -126,6 +126,10 @@ __global__ void k_bfs_init(int32_t *levels, uint32_t V, uint32_t root) {
     levels[v] = (v == root) ? 0 : -1;
 }
 
+__global__ void k_bfs_set_bit(uint32_t *bm, uint32_t v) {
+  if (threadIdx.x == 0) bm[v >> 5] |= 1u << (v & 31);
+}
+
 // frontier of depth d: bitmap words written whole by one lane per 32 vertices; size into *F
 // (one atomic per CTA)
 __global__ void k_bfs_frontier(const int32_t *__restrict__ levels, uint32_t V, int32_t d,
@@ -176,6 +180,23 @@ __global__ void k_bfs_rowlen(const uint32_t *__restrict__ frontier, uint32_t F,
   }
 }
 
+// Discovery of v at `depth`.  With a next-frontier bitmap (single-store BFS) the first
+// discoverer also sets v's bit and counts it, so the next level needs no sweep over `levels`
+// to find its frontier.  Racing discoverers all store the same depth; the atomicOr's old
+// value picks exactly one of them for the count.
+__device__ __forceinline__ uint32_t bfs_discover(int32_t *levels, uint32_t v, int32_t depth, uint32_t *bm_next) {
+  if (levels[v] != -1) return 0;
+  levels[v] = depth;
+  if (!bm_next) return 0;
+  const uint32_t bit = 1u << (v & 31);
+  return (atomicOr(bm_next + (v >> 5), bit) & bit) ? 0u : 1u;
+}
+
+__device__ __forceinline__ void bfs_count(uint32_t found, uint32_t *fnext) {
+  found = __reduce_add_sync(0xffffffffu, found);
+  if ((threadIdx.x & 31) == 0 && found) atomicAdd(fnext, found);
+}
+
 // Sparse levels -- Neighbour Gathering over the concatenated frontier rows (Alg. 3),
 // load-balanced: warp w owns the contiguous slot range [w*C, (w+1)*C) of the concatenation,
 // binary-searches its first row once, then walks forward 32 slots at a time.
@@ -184,7 +205,8 @@ __global__ void __launch_bounds__(TA) k_bfs_expand(const uint32_t *__restrict__ 
                                                    const uint64_t *__restrict__ row_offset,
                                                    const uint64_t *__restrict__ key,
                                                    const uint32_t *__restrict__ tmask, uint32_t L,
-                                                   int32_t *levels, int32_t depth, uint32_t rb) {
+                                                   int32_t *levels, int32_t depth, uint32_t rb,
+                                                   uint32_t *bm_next, uint32_t *fnext) {
   const int lane = threadIdx.x & 31;
   const uint64_t total = off[F];
   const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
@@ -195,6 +217,7 @@ __global__ void __launch_bounds__(TA) k_bfs_expand(const uint32_t *__restrict__ 
   uint32_t i0 = 0;
   if (lane == 0) i0 = upper_bound_u64(off, 0, F + 1, beg) - 1;
   i0 = __shfl_sync(0xffffffffu, i0, 0);
+  uint32_t found = 0;
   for (uint64_t base = beg; base < end; base += 32) {
     const uint64_t gi = base + lane;
     uint32_t i = i0;
@@ -203,36 +226,69 @@ __global__ void __launch_bounds__(TA) k_bfs_expand(const uint32_t *__restrict__ 
       uint32_t u = frontier[i] - rb;
       uint64_t s = row_offset[u] + (gi - off[i]);
       uint64_t k;
-      if (edge_at(key, tmask, L, s, &k)) {
-        uint32_t v = (uint32_t)k;
-        if (levels[v] == -1) levels[v] = depth;
-      }
+      if (edge_at(key, tmask, L, s, &k)) found += bfs_discover(levels, (uint32_t)k, depth, bm_next);
     }
     i0 = __shfl_sync(0xffffffffu, i, 31);
   }
+  if (fnext) bfs_count(found, fnext);
 }
 
 // A leaf is active when its source range holds a frontier vertex.  The range comes from the
 // locate heads (every vertex has a guard, so a leaf spans at most L sources).
-__global__ void k_bfs_leaf_active(const uint64_t *__restrict__ head, uint64_t nleaves, uint32_t V,
-                                  const uint32_t *__restrict__ bm, uint32_t *__restrict__ act) {
-  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
-       l += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t h0 = head[l], h1 = l + 1 < nleaves ? head[l + 1] : KEY_NONE;
-    uint32_t ua = h0 == KEY_NONE ? V : (uint32_t)(h0 >> 32);
-    uint32_t ub = h1 == KEY_NONE ? V - 1 : (uint32_t)(h1 >> 32);
-    uint32_t a = 0;
-    for (uint32_t u = ua; u <= ub && u < V; ++u)
-      if ((__ldg(bm + (u >> 5)) >> (u & 31)) & 1u) { a = 1; break; }
-    act[l] = a;
+// Active leaves appended to alist: a CTA tests 4 x 256 consecutive leaves (head loads first,
+// then the bitmap probes), ranks them with ballots + a 32-entry CTA scan and reserves its
+// slots with ONE atomic.  The CTA order in alist does not matter to the sweep.
+constexpr int BFS_LA_K = 4;
+__global__ void __launch_bounds__(TA) k_bfs_leaf_active(const uint64_t *__restrict__ head, uint64_t nleaves,
+                                                        uint32_t V, const uint32_t *__restrict__ bm,
+                                                        uint32_t *__restrict__ alist, uint32_t *__restrict__ nact) {
+  static_assert(BFS_LA_K * (TA / 32) == 32, "one warp scans the per-warp counts");
+  __shared__ uint32_t wofs[BFS_LA_K * (TA / 32)];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint64_t per = (uint64_t)TA * BFS_LA_K;
+  for (uint64_t b0 = blockIdx.x * per; b0 < nleaves; b0 += (uint64_t)gridDim.x * per) {
+    uint64_t h0[BFS_LA_K], h1[BFS_LA_K];
+#pragma unroll
+    for (int k = 0; k < BFS_LA_K; ++k) {
+      const uint64_t l = b0 + k * TA + threadIdx.x;
+      h0[k] = l < nleaves ? head[l] : KEY_NONE;
+      h1[k] = l + 1 < nleaves ? head[l + 1] : KEY_NONE;
+    }
+    uint32_t act[BFS_LA_K], bal[BFS_LA_K];
+#pragma unroll
+    for (int k = 0; k < BFS_LA_K; ++k) {
+      act[k] = 0;
+      if (h0[k] != KEY_NONE) {
+        const uint32_t ua = (uint32_t)(h0[k] >> 32);
+        const uint32_t ub = h1[k] == KEY_NONE ? V - 1 : (uint32_t)(h1[k] >> 32);
+        for (uint32_t u = ua; u <= ub && u < V; ++u)
+          if ((__ldg(bm + (u >> 5)) >> (u & 31)) & 1u) { act[k] = 1; break; }
+      }
+      bal[k] = __ballot_sync(0xffffffffu, act[k]);
+      if (lane == 0) wofs[k * (TA / 32) + warp] = __popc(bal[k]);
+    }
+    __syncthreads();
+    if (threadIdx.x < 32) {                         // exclusive scan of the 32 warp counts
+      const uint32_t v = wofs[threadIdx.x];
+      uint32_t x = v;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+        if (lane >= o) x += y;
+      }
+      const uint32_t tot = __shfl_sync(0xffffffffu, x, 31);
+      uint32_t base = 0;
+      if (lane == 0 && tot) base = atomicAdd(nact, tot);
+      base = __shfl_sync(0xffffffffu, base, 0);
+      wofs[threadIdx.x] = base + x - v;
+    }
+    __syncthreads();
+    const uint32_t lt = (1u << lane) - 1u;
+#pragma unroll
+    for (int k = 0; k < BFS_LA_K; ++k)
+      if (act[k]) alist[wofs[k * (TA / 32) + warp] + __popc(bal[k] & lt)] = (uint32_t)(b0 + k * TA + threadIdx.x);
+    __syncthreads();
   }
-}
-
-__global__ void k_bfs_leaf_list(const uint32_t *__restrict__ act, const uint32_t *__restrict__ apos,
-                                uint64_t nleaves, uint32_t *__restrict__ alist) {
-  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nleaves;
-       l += (uint64_t)gridDim.x * blockDim.x)
-    if (act[l]) alist[apos[l]] = (uint32_t)l;
 }
 
 // Dense levels: sweep the active leaves, two groups of 4 slots per thread, expanding the
@@ -242,8 +298,9 @@ __global__ void __launch_bounds__(TA) k_bfs_sweep(const uint64_t *__restrict__ k
                                                   const uint32_t *__restrict__ alist,
                                                   const uint32_t *__restrict__ nact_p,
                                                   const uint32_t *__restrict__ bm, int32_t *levels,
-                                                  int32_t depth) {
+                                                  int32_t depth, uint32_t *bm_next, uint32_t *fnext) {
   const uint32_t tpl = L / 4;
+  uint32_t found = 0;
   const uint64_t n4 = (uint64_t)(*nact_p) * tpl;
   for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4;
        t += (uint64_t)gridDim.x * blockDim.x) {
@@ -254,9 +311,10 @@ __global__ void __launch_bounds__(TA) k_bfs_sweep(const uint64_t *__restrict__ k
       if (!edge4(sl, j)) continue;
       uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
       if (!((__ldg(bm + (u >> 5)) >> (u & 31)) & 1u)) continue;
-      if (levels[v] == -1) levels[v] = depth;
+      found += bfs_discover(levels, v, depth, bm_next);
     }
   }
+  if (fnext) bfs_count(found, fnext);
 }
 
 constexpr uint32_t BFS_SPARSE_F = 4096;   // frontiers up to this size use row expansion
@@ -267,25 +325,46 @@ gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
   return GPMA_OK;
 }
 
-// One BFS level: the frontier is {v : levels[v] == depth-1} (levels may be replicated across
-// shards); the owned rows of the frontier are expanded and newly reached vertices get
-// `depth`.  *frontier = the frontier size (0: the traversal is over, nothing expanded).
-gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontier, cudaStream_t s) {
-  Scratch &X = g->an[AN_BFS];
-  ScanScope scan_scope_(X.scan);
+// Expand the frontier bitmap `bm` (F vertices) by one level: sparse -- row expansion over the
+// frontier list; dense -- sweep of the active leaves.  Discoveries get `depth`; with bm_next
+// they are also marked there and counted into *fnext (device).
+static gpma_status bfs_expand_level(gpma *g, Scratch &X, int32_t *levels, int32_t depth, const uint32_t *bm,
+                                    uint32_t F, uint32_t *bm_next, uint32_t *fnext, cudaStream_t s) {
   const uint64_t V = g->V, nl = g->cap / g->L;
   GP_CHECK(g, ensure(X.b[0], (V + 1) * 4, s));
-  GP_CHECK(g, ensure(X.b[2], (std::max<uint64_t>(V, nl) + 2) * 8, s));
-  GP_CHECK(g, ensure(X.b[3], (V / 32 + 2) * 4, s));
+  GP_CHECK(g, ensure(X.b[2], ((uint64_t)BFS_SPARSE_F + 2) * 8, s));
   GP_CHECK(g, ensure(X.misc, (nl + 2) * 4, s));
   uint32_t *list = (uint32_t *)X.b[0].p;
   uint64_t *off = (uint64_t *)X.b[2].p;
-  uint32_t *act = (uint32_t *)X.b[2].p;          // shares off's buffer: never both in a level
-  uint32_t *apos = act + nl + 1;
   uint32_t *alist = (uint32_t *)X.misc.p;
+  uint32_t *cnt_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum2);   // list / active-leaf count
+  const uint32_t *tmask = tmask_of(g);
+  GP_CHECK(g, cudaMemsetAsync(cnt_d, 0, 4, s));
+  if (F <= BFS_SPARSE_F) {
+    GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, cnt_d);
+    GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, g->rb, g->nr, off);
+    scan_u64(g, off, off, F, s);
+    GP_LAUNCH(g, k_bfs_expand, grid_cap(), TA, 0, s, list, F, off, g->row_offset, g->key, tmask, g->L,
+              levels, depth, g->rb, bm_next, fnext);
+  } else {
+    GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, alist, cnt_d);
+    GP_LAUNCH(g, k_bfs_sweep, grid_cap(), TA, 0, s, g->key, tmask, g->L, alist, cnt_d, bm, levels, depth,
+              bm_next, fnext);
+  }
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+// One BFS level of a (possibly sharded) store: the frontier is {v : levels[v] == depth-1}
+// (levels may be replicated across shards); the owned rows of the frontier are expanded and
+// newly reached vertices get `depth`.  *frontier = the frontier size (0: nothing expanded).
+gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontier, cudaStream_t s) {
+  Scratch &X = g->an[AN_BFS];
+  ScanScope scan_scope_(X.scan);
+  const uint64_t V = g->V;
+  GP_CHECK(g, ensure(X.b[3], (V / 32 + 2) * 4, s));
   uint32_t *bm = (uint32_t *)X.b[3].p;
   uint32_t *F_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum);
-  const uint32_t *tmask = tmask_of(g);
   GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
   GP_LAUNCH(g, k_bfs_frontier, grid_for(V), TA, 0, s, levels, (uint32_t)V, depth - 1, bm, F_d);
   GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
@@ -293,32 +372,34 @@ gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontie
   const uint32_t F = (uint32_t)(X.ctrl_h->sum & 0xFFFFFFFFu);
   *frontier = F;
   if (!F) return GPMA_OK;
-  if (F <= BFS_SPARSE_F) {
-    GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
-    GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, F_d);
-    GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, g->rb, g->nr, off);
-    scan_u64(g, off, off, F, s);
-    GP_LAUNCH(g, k_bfs_expand, grid_cap(), TA, 0, s, list, F, off, g->row_offset, g->key, tmask, g->L,
-              levels, depth, g->rb);
-  } else {
-    GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, act);
-    scan_u32(g, act, apos, nl, s);
-    GP_LAUNCH(g, k_bfs_leaf_list, grid_for(nl), TA, 0, s, act, apos, nl, alist);
-    GP_LAUNCH(g, k_bfs_sweep, grid_cap(), TA, 0, s, g->key, tmask, g->L, alist, apos + nl, bm, levels,
-              depth);
-  }
-  GP_CHECK(g, cudaGetLastError());
-  return GPMA_OK;
+  return bfs_expand_level(g, X, levels, depth, bm, F, nullptr, nullptr, s);
 }
 
+// Whole-store BFS (Alg. 3 level by level): each level's discoveries build the next frontier
+// bitmap directly; one host read of the frontier size per level.
 gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
-  gpma_status st = bfs_init(g, root, levels, s);
-  for (int32_t depth = 1; st == GPMA_OK; ++depth) {
-    uint32_t F = 0;
-    st = bfs_level(g, levels, depth, &F, s);
-    if (!F) break;
+  Scratch &X = g->an[AN_BFS];
+  ScanScope scan_scope_(X.scan);
+  const uint64_t V = g->V, words = (V + 31) / 32 + 1;
+  GP_CHECK(g, ensure(X.b[3], words * 4, s));
+  GP_CHECK(g, ensure(X.b[1], words * 4, s));
+  uint32_t *bm[2] = {(uint32_t *)X.b[3].p, (uint32_t *)X.b[1].p};
+  uint32_t *F_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum);
+  GP_CHECK(g, cudaMemsetAsync(bm[0], 0, words * 4, s));
+  GP_LAUNCH(g, k_bfs_init, grid_for(V), TA, 0, s, levels, g->V, root);
+  GP_LAUNCH(g, k_bfs_set_bit, 1, 32, 0, s, bm[0], root);
+  uint32_t F = 1;
+  int cur = 0;
+  for (int32_t depth = 1; F; ++depth, cur ^= 1) {
+    GP_CHECK(g, cudaMemsetAsync(bm[cur ^ 1], 0, words * 4, s));
+    GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
+    gpma_status st = bfs_expand_level(g, X, levels, depth, bm[cur], F, bm[cur ^ 1], F_d, s);
+    if (st) return st;
+    GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, cudaStreamSynchronize(s));
+    F = (uint32_t)(X.ctrl_h->sum & 0xFFFFFFFFu);
   }
-  return st;
+  return GPMA_OK;
 }
 
 // ------------------------------------------------------------------ CC
