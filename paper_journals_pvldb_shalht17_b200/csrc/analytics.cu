@@ -496,6 +496,34 @@ __global__ void __launch_bounds__(TA) k_cc_sample(const uint64_t *__restrict__ k
   }
 }
 
+// Sample round over the rows (guard-indexed stores): each owned row hooks its first NS live
+// edges, found from row_offset (R8) -- slot row_offset[u] + 1 follows guard u-1 -- instead
+// of sweeping every slot; the scan skips a leaf's empty tail and stops at guard u.
+template <bool H, int NS>
+__global__ void __launch_bounds__(TA) k_cc_sample_rows(const uint64_t *__restrict__ key,
+                                                       const uint32_t *__restrict__ tmask,
+                                                       const uint64_t *__restrict__ row_offset, uint32_t L,
+                                                       uint32_t nr, uint32_t rb, uint32_t *p) {
+  const uint64_t pol = H ? l2_evict_last_policy() : 0;
+  for (uint64_t r = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; r < nr; r += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t sl = r ? row_offset[r] + 1 : 0;
+    const uint64_t e = row_offset[r + 1];
+    const uint32_t u = (uint32_t)r + rb;
+    int found = 0;
+    for (int it = 0; sl < e && found < NS && it < 64; ++it, ++sl) {
+      const uint64_t k = __ldcs(key + sl);
+      if (k == KEY_NONE) {                 // empty tail of a leaf: continue at the next leaf
+        sl |= (uint64_t)(L - 1);
+        continue;
+      }
+      if ((__ldg(tmask + sl / L) >> (uint32_t)(sl % L)) & 1u) continue;   // tombstone
+      const uint32_t v = (uint32_t)k;
+      ++found;
+      if (u != v && cc_ld<H>(p + u, pol) != cc_ld<H>(p + v, pol)) cc_hook<H>(p, u, v, pol);
+    }
+  }
+}
+
 __global__ void k_cc_compress(uint32_t *p, uint32_t V) {
   for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
        v += (uint64_t)gridDim.x * blockDim.x) {
@@ -546,6 +574,29 @@ static int cc_hint() {
   return v;
 }
 
+// sampled first round: row based when every row has its guard (GPMA_CC_SAMPLE=0 forces the
+// slot sweep), else the (source, leaf)-run sweep
+static int cc_sample_mode() {
+  static const int v = [] { const char *e = getenv("GPMA_CC_SAMPLE"); return e ? atoi(e) : 2; }();
+  return v;
+}
+
+static cudaError_t cc_sample(gpma *g, uint32_t *p, cudaStream_t s) {
+  const uint32_t *tmask = tmask_of(g);
+  const int m = cc_sample_mode();
+  if (g->rows_indexed && m > 0) {
+    if (m == 1) GP_LAUNCH(g, (k_cc_sample_rows<true, 1>), grid_for(g->nr, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->row_offset, g->L,
+                          g->nr, g->rb, p);
+    else GP_LAUNCH(g, (k_cc_sample_rows<true, 2>), grid_for(g->nr, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->row_offset, g->L,
+                   g->nr, g->rb, p);
+  } else if (cc_hint()) {
+    GP_LAUNCH(g, k_cc_sample<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
+  } else {
+    GP_LAUNCH(g, k_cc_sample<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
+  }
+  return cudaGetLastError();
+}
+
 __global__ void k_cc_final(uint32_t *p, uint32_t *labels, uint32_t V) {
   for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
        v += (uint64_t)gridDim.x * blockDim.x) {
@@ -577,8 +628,7 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
   const uint32_t *tmask = tmask_of(g);
   if (init) GP_LAUNCH(g, k_cc_init, grid_for(V), TA, 0, s, labels, g->V);
   GP_CHECK(g, cudaMemcpyAsync(prev, labels, V * 4, cudaMemcpyDeviceToDevice, s));
-  if (cc_hint()) GP_LAUNCH(g, k_cc_sample<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
-  else GP_LAUNCH(g, k_cc_sample<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, labels);
+  GP_CHECK(g, cc_sample(g, labels, s));
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
   if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
   else GP_LAUNCH(g, k_cc_hook<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
@@ -599,8 +649,7 @@ gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s) {
   uint32_t *p = (uint32_t *)X.b[0].p;
   const uint32_t *tmask = tmask_of(g);
   GP_LAUNCH(g, k_cc_init, grid_for(g->V), TA, 0, s, p, g->V);
-  if (cc_hint()) GP_LAUNCH(g, k_cc_sample<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
-  else GP_LAUNCH(g, k_cc_sample<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->cap, g->L, p);
+  GP_CHECK(g, cc_sample(g, p, s));
   GP_LAUNCH(g, k_cc_compress, grid_for(g->V), TA, 0, s, p, g->V);
   if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
   else GP_LAUNCH(g, k_cc_hook<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);

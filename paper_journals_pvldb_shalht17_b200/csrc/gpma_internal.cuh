@@ -142,6 +142,8 @@ struct ScanScope {
 
 // grid cap of the grid-stride kernels (default MAX_RESIDENT_BLOCKS; GPMA_GRID_CAP overrides)
 int grid_cap();
+// SMs of the current device (persistent sweeps launch one CTA per SM)
+int num_sms();
 
 inline unsigned grid_for(uint64_t n, int block = 256, int max_blocks = 0) {
   if (max_blocks <= 0) max_blocks = grid_cap();

@@ -76,6 +76,16 @@ int grid_cap() {
   return v;
 }
 
+int num_sms() {
+  static const int v = [] {
+    int d = 0, n = 0;
+    cudaGetDevice(&d);
+    cudaDeviceGetAttribute(&n, cudaDevAttrMultiProcessorCount, d);
+    return n > 0 ? n : 148;
+  }();
+  return v;
+}
+
 void set_err(gpma *g, const std::string &msg) {
   std::lock_guard<std::mutex> lk(g->mu);
   g->err = msg;
