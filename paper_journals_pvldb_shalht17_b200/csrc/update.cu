@@ -237,14 +237,18 @@ __global__ void __launch_bounds__(256) k_level0(const uint64_t *__restrict__ pk,
         uk = pk[j0 + sl];
         uv = pv[j0 + sl];
       }
+      // merged ranks: one round per update of the sub-warp (u <= max_0 when accepted; most
+      // accepted leaves take a single update), the leaf side by one ballot per round
       uint32_t below_u = 0, below_l = 0;
       bool drop = false;
-      for (uint32_t i = 0; i < L; ++i) {                // merged ranks (width-L shuffles)
+      const uint32_t umax = __reduce_max_sync(0xffffffffu, ok ? u : 0u);
+      for (uint32_t i = 0; i < umax; ++i) {
+        const bool vi = ok && i < u;                    // uniform within the sub-warp
         const uint64_t ui = __shfl_sync(0xffffffffu, uk, i, L);
-        const uint64_t ki = __shfl_sync(0xffffffffu, ks, i, L);
-        below_u += i < u && ui < ks;
-        below_l += ((lbits >> i) & 1u) && ki < uk;
-        drop |= !ins && live && i < u && ui == ks;
+        below_u += vi && ui < ks;
+        const uint32_t bl = __popc((__ballot_sync(0xffffffffu, vi && live && ks < ui) & submask) >> (sub * L));
+        if (sl == i) below_l = bl;
+        drop |= !ins && live && vi && ui == ks;
       }
       const uint32_t N = ins ? n + u : n - u;
       const uint32_t live_rank = __popc(lbits & below_me);
