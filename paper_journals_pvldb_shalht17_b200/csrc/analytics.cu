@@ -113,7 +113,7 @@ __global__ void __launch_bounds__(TA) k_deg_count(const uint64_t *__restrict__ k
 }
 
 gpma_status recompute_degrees(gpma *g, cudaStream_t s) {
-  GP_CHECK(g, cudaMemsetAsync(g->deg, 0, (uint64_t)g->nr * 4, s));
+  GP_CHECK(g, fill_zero(g, g->deg, (uint64_t)g->nr * 4, s));
   GP_LAUNCH(g, k_deg_count, grid_for(g->cap / 4), TA, 0, s, g->key, tmask_of(g), g->L, g->cap, g->deg, g->rb);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
@@ -317,7 +317,11 @@ __global__ void __launch_bounds__(TA) k_bfs_sweep(const uint64_t *__restrict__ k
   if (fnext) bfs_count(found, fnext);
 }
 
-constexpr uint32_t BFS_SPARSE_F = 4096;   // frontiers up to this size use row expansion
+// frontiers up to this size use row expansion (GPMA_BFS_SPARSE overrides)
+static uint32_t bfs_sparse_f() {
+  static const uint32_t v = [] { const char *e = getenv("GPMA_BFS_SPARSE"); return e ? (uint32_t)atol(e) : 32768u; }();
+  return v;
+}
 
 gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
   GP_LAUNCH(g, k_bfs_init, grid_for(g->V), TA, 0, s, levels, g->V, root);
@@ -332,15 +336,15 @@ static gpma_status bfs_expand_level(gpma *g, Scratch &X, int32_t *levels, int32_
                                     uint32_t F, uint32_t *bm_next, uint32_t *fnext, cudaStream_t s) {
   const uint64_t V = g->V, nl = g->cap / g->L;
   GP_CHECK(g, ensure(X.b[0], (V + 1) * 4, s));
-  GP_CHECK(g, ensure(X.b[2], ((uint64_t)BFS_SPARSE_F + 2) * 8, s));
   GP_CHECK(g, ensure(X.misc, (nl + 2) * 4, s));
   uint32_t *list = (uint32_t *)X.b[0].p;
-  uint64_t *off = (uint64_t *)X.b[2].p;
   uint32_t *alist = (uint32_t *)X.misc.p;
   uint32_t *cnt_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum2);   // list / active-leaf count
   const uint32_t *tmask = tmask_of(g);
-  GP_CHECK(g, cudaMemsetAsync(cnt_d, 0, 4, s));
-  if (F <= BFS_SPARSE_F) {
+  GP_CHECK(g, fill_zero(g, cnt_d, 4, s));
+  if (F <= bfs_sparse_f()) {
+    GP_CHECK(g, ensure(X.b[2], ((uint64_t)bfs_sparse_f() + 2) * 8, s));   // fixed size: no regrowth per level
+    uint64_t *off = (uint64_t *)X.b[2].p;
     GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, cnt_d);
     GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, g->rb, g->nr, off);
     scan_u64(g, off, off, F, s);
@@ -365,9 +369,9 @@ gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontie
   GP_CHECK(g, ensure(X.b[3], (V / 32 + 2) * 4, s));
   uint32_t *bm = (uint32_t *)X.b[3].p;
   uint32_t *F_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum);
-  GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
+  GP_CHECK(g, fill_zero(g, F_d, 4, s));
   GP_LAUNCH(g, k_bfs_frontier, grid_for(V), TA, 0, s, levels, (uint32_t)V, depth - 1, bm, F_d);
-  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, readback(g, &X.ctrl_h->sum, F_d, 4, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   const uint32_t F = (uint32_t)(X.ctrl_h->sum & 0xFFFFFFFFu);
   *frontier = F;
@@ -385,17 +389,17 @@ gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
   GP_CHECK(g, ensure(X.b[1], words * 4, s));
   uint32_t *bm[2] = {(uint32_t *)X.b[3].p, (uint32_t *)X.b[1].p};
   uint32_t *F_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum);
-  GP_CHECK(g, cudaMemsetAsync(bm[0], 0, words * 4, s));
+  GP_CHECK(g, fill_zero(g, bm[0], words * 4, s));
   GP_LAUNCH(g, k_bfs_init, grid_for(V), TA, 0, s, levels, g->V, root);
   GP_LAUNCH(g, k_bfs_set_bit, 1, 32, 0, s, bm[0], root);
   uint32_t F = 1;
   int cur = 0;
   for (int32_t depth = 1; F; ++depth, cur ^= 1) {
-    GP_CHECK(g, cudaMemsetAsync(bm[cur ^ 1], 0, words * 4, s));
-    GP_CHECK(g, cudaMemsetAsync(F_d, 0, 4, s));
+    GP_CHECK(g, fill_zero(g, bm[cur ^ 1], words * 4, s));
+    GP_CHECK(g, fill_zero(g, F_d, 4, s));
     gpma_status st = bfs_expand_level(g, X, levels, depth, bm[cur], F, bm[cur ^ 1], F_d, s);
     if (st) return st;
-    GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, F_d, 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, readback(g, &X.ctrl_h->sum, F_d, 4, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
     F = (uint32_t)(X.ctrl_h->sum & 0xFFFFFFFFu);
   }
@@ -633,9 +637,9 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
   if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
   else GP_LAUNCH(g, k_cc_hook<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
-  GP_CHECK(g, cudaMemsetAsync(&X.ctrl_d->sum, 0, 8, s));
+  GP_CHECK(g, fill_zero(g, &X.ctrl_d->sum, 8, s));
   GP_LAUNCH(g, k_cc_changed, grid_for(V), TA, 0, s, labels, prev, g->V, X.ctrl_d);
-  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, &X.ctrl_d->sum, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, readback(g, &X.ctrl_h->sum, &X.ctrl_d->sum, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   *changed = X.ctrl_h->sum;
   GP_CHECK(g, cudaGetLastError());
@@ -833,15 +837,32 @@ __global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ 
   __shared__ double red[32];
   const T base = (T(1) - d) / T(V) + d * T(*dsum_in / (double)V);
   double e = 0, dl = 0;
-  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
-       v += (uint64_t)gridDim.x * blockDim.x) {
-    T nx = base + d * PrAcc<T>::dec(y[v]);
-    e += fabs((double)nx - (double)x[v]);
-    x[v] = nx;
-    y[v] = 0;
-    uint32_t dg = deg[v];
-    contrib[v] = PrAcc<T>::enc(dg ? nx / T(dg) : T(0));
-    if (!dg) dl += (double)nx;
+  constexpr int PU = 4;                                  // 4 vertices in flight per thread
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t v0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v0 < V; v0 += PU * stride) {
+    typename PrAcc<T>::A yo[PU];
+    T xo[PU];
+    uint32_t dg[PU];
+#pragma unroll
+    for (int j = 0; j < PU; ++j) {
+      const uint64_t v = v0 + j * stride;
+      if (v < V) {
+        yo[j] = __ldcs(y + v);
+        xo[j] = __ldcs(x + v);
+        dg[j] = __ldcs(deg + v);
+      }
+    }
+#pragma unroll
+    for (int j = 0; j < PU; ++j) {
+      const uint64_t v = v0 + j * stride;
+      if (v >= V) continue;
+      const T nx = base + d * PrAcc<T>::dec(yo[j]);
+      e += fabs((double)nx - (double)xo[j]);
+      x[v] = nx;
+      y[v] = 0;
+      contrib[v] = PrAcc<T>::enc(dg[j] ? nx / T(dg[j]) : T(0));
+      if (!dg[j]) dl += (double)nx;
+    }
   }
   double se = block_sum_d(e, red);
   double sd = block_sum_d(dl, red);
@@ -882,7 +903,7 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   A *contrib = (A *)X.b[1].p, *y = (A *)X.b[2].p;
   double *acc = (double *)X.b[3].p;   // [0],[1] dangling ping-pong, [2] error
   const uint32_t passes = pr_passes(V * sizeof(A));
-  GP_CHECK(g, cudaMemsetAsync(acc, 0, 4 * sizeof(double), s));
+  GP_CHECK(g, fill_zero(g, acc, 4 * sizeof(double), s));
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
   int it = 0, cur = 0;
   while (it < max_iter) {
@@ -891,13 +912,13 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
       GP_LAUNCH(g, (k_pr_push_win<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
                 g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes),
                 pr_hint());
-    GP_CHECK(g, cudaMemsetAsync(acc + 2, 0, sizeof(double), s));
-    GP_CHECK(g, cudaMemsetAsync(acc + (cur ^ 1), 0, sizeof(double), s));
+    GP_CHECK(g, fill_zero(g, acc + 2, sizeof(double), s));
+    GP_CHECK(g, fill_zero(g, acc + (cur ^ 1), sizeof(double), s));
     GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
               acc + (cur ^ 1), acc + 2);
     cur ^= 1;
     ++it;
-    GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum2, acc + 2, 8, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, readback(g, &X.ctrl_h->sum2, acc + 2, 8, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
     double e;
     memcpy(&e, &X.ctrl_h->sum2, 8);
@@ -969,10 +990,10 @@ gpma_status pr_update(gpma *g, double *x, uint64_t *y, double d, double *err, cu
   Scratch &X = g->an[AN_PR];
   ScanScope scan_scope_(X.scan);
   double *e_d = reinterpret_cast<double *>(&X.ctrl_d->sum2);
-  GP_CHECK(g, cudaMemsetAsync(e_d, 0, 8, s));
+  GP_CHECK(g, fill_zero(g, e_d, 8, s));
   GP_LAUNCH(g, k_prd_update, grid_for(g->V), TA, 0, s, x, (unsigned long long *)y, g->V, d, e_d);
-  GP_CHECK(g, cudaMemsetAsync(y + g->V, 0, 8, s));
-  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum2, e_d, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, fill_zero(g, y + g->V, 8, s));
+  GP_CHECK(g, readback(g, &X.ctrl_h->sum2, e_d, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   memcpy(err, &X.ctrl_h->sum2, 8);
   GP_CHECK(g, cudaGetLastError());
@@ -1062,7 +1083,7 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
   uint64_t *lc = (uint64_t *)X.lpre.p;
   GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gcnt_of(g), nl, lc);
   scan_u64(g, lc, lc, nl, s);
-  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, lc + nl, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, readback(g, &X.ctrl_h->sum, lc + nl, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   uint64_t nnz = X.ctrl_h->sum;
   if (nnz_out) *nnz_out = nnz;
@@ -1071,7 +1092,7 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
     set_err(g, "export_csr: nnz_capacity too small");
     return GPMA_ERR_INVALID_ARG;
   }
-  GP_CHECK(g, cudaMemsetAsync(row_ptr, 0, 8, s));
+  GP_CHECK(g, fill_zero(g, row_ptr, 8, s));
   GP_LAUNCH(g, k_exp_write, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, g->val, tmask_of(g), g->L, g->cap, lc,
             row_ptr, col, val, g->rb);
   GP_CHECK(g, cudaGetLastError());

@@ -109,7 +109,25 @@ gpma_status apply_config(gpma *g, const gpma_config *cfg, uint32_t *leaf, uint64
 
 void free_handle(gpma *g);
 
+// Keep freed stream-ordered blocks in the device's default pool across synchronisations (the
+// default release threshold 0 returns them to the OS at every sync, so each regrowth of a
+// scratch buffer would map memory again).
+static void keep_pool_memory() {
+  static const bool done = [] {
+    int d = 0;
+    cudaMemPool_t pool;
+    if (cudaGetDevice(&d) == cudaSuccess && cudaDeviceGetDefaultMemPool(&pool, d) == cudaSuccess) {
+      uint64_t thr = ~0ull;
+      cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr);
+    }
+    cudaGetLastError();
+    return true;
+  }();
+  (void)done;
+}
+
 gpma *new_handle(uint32_t V) {
+  keep_pool_memory();
   gpma *g = new (std::nothrow) gpma();
   if (!g) return nullptr;
   g->V = V;
@@ -243,7 +261,7 @@ gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t l
     }
   }
   if (st == GPMA_OK) {
-    cudaMemsetAsync(g->row_offset, 0, ((uint64_t)g->nr + 1) * 8, s);
+    gp::fill_zero(g, g->row_offset, ((uint64_t)g->nr + 1) * 8, s);
     st = gp::load_raw(g, keys, vals, s);
   }
   if (st == GPMA_OK && cudaStreamSynchronize(s) != cudaSuccess) st = GPMA_ERR_CUDA;

@@ -26,9 +26,9 @@ gpma_status route(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t 
   uint64_t *k0 = (uint64_t *)g->b_stage[2].p;
   uint32_t *v0 = (uint32_t *)g->b_stage[3].p;
   uint64_t *starts = (uint64_t *)((char *)g->b_stage[3].p + ((n * 4 + 7) & ~7ull));
-  GP_CHECK(g, cudaMemcpyAsync(k0, keys, n * 8, cudaMemcpyDefault, s));
-  if (vals) GP_CHECK(g, cudaMemcpyAsync(v0, vals, n * 4, cudaMemcpyDefault, s));
-  else GP_CHECK(g, cudaMemsetAsync(v0, 0, n * 4, s));
+  GP_CHECK(g, stage_in(g, k0, keys, n * 8, s));
+  if (vals) GP_CHECK(g, stage_in(g, v0, vals, n * 4, s));
+  else GP_CHECK(g, fill_zero(g, v0, n * 4, s));
   gpma_status st = radix_partition_owner(g, k0, v0, out_keys, out_vals, n, div, nranks, starts, s);
   if (st) return st;
   std::vector<uint64_t> h(nranks + 1);

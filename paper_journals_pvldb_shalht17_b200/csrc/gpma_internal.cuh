@@ -142,6 +142,13 @@ struct ScanScope {
 
 // grid cap of the grid-stride kernels (default MAX_RESIDENT_BLOCKS; GPMA_GRID_CAP overrides)
 int grid_cap();
+// copy `bytes` (multiple of 4, 4-B aligned) from device memory to PINNED host memory with a
+// kernel (no copy engine); stream-ordered like cudaMemcpyAsync
+cudaError_t readback(gpma *g, void *host_pinned, const void *dev, size_t bytes, cudaStream_t s);
+// copy a caller's input (host or device pointer) into library scratch, stream-ordered
+cudaError_t stage_in(gpma *g, void *dst, const void *src, size_t bytes, cudaStream_t s);
+// zero `bytes` (multiple of 4, 4-B aligned) of device memory with a kernel, stream-ordered
+cudaError_t fill_zero(gpma *g, void *dst, size_t bytes, cudaStream_t s);
 // SMs of the current device (persistent sweeps launch one CTA per SM)
 int num_sms();
 

@@ -76,6 +76,79 @@ int grid_cap() {
   return v;
 }
 
+// Small device -> pinned-host read-backs by a one-warp kernel (zero-copy stores over the bus)
+// instead of cudaMemcpyAsync: a DMA read-back queues on the D2H copy engine behind whatever a
+// user's copy stream is moving (e.g. the Fig. 2 pipeline's result transfers), which would
+// stall every host round trip of the library for the length of that transfer.
+__global__ void k_readback(uint32_t *dst, const uint32_t *__restrict__ src, uint32_t nwords) {
+  for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) dst[i] = src[i];
+}
+
+cudaError_t readback(gpma *g, void *host_pinned, const void *dev, size_t bytes, cudaStream_t s) {
+  g->launches++;
+  k_readback<<<1, 32, 0, s>>>((uint32_t *)host_pinned, (const uint32_t *)dev, (uint32_t)(bytes / 4));
+  return cudaGetLastError();
+}
+
+// Staging copy of a caller's batch into library scratch: a kernel when the source is device
+// memory (same reason as readback: a D2D cudaMemcpyAsync may wait on a busy copy engine), a
+// DMA copy when it is host memory.  bytes % 4 == 0, 4-B aligned.
+__global__ void k_copy_words(uint32_t *__restrict__ dst, const uint32_t *__restrict__ src, uint64_t nwords,
+                             int vec4) {
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
+  uint64_t head = 0;
+  if (vec4) {
+    const uint64_t n4 = nwords / 4;
+    for (uint64_t i = i0; i < n4; i += stride)
+      reinterpret_cast<uint4 *>(dst)[i] = __ldcs(reinterpret_cast<const uint4 *>(src) + i);
+    head = n4 * 4;
+  }
+  for (uint64_t i = head + i0; i < nwords; i += stride) dst[i] = src[i];
+}
+
+cudaError_t stage_in(gpma *g, void *dst, const void *src, size_t bytes, cudaStream_t s) {
+  if (!bytes) return cudaSuccess;
+  cudaPointerAttributes a{};
+  cudaError_t e = cudaPointerGetAttributes(&a, src);
+  if (e != cudaSuccess) {
+    cudaGetLastError();   // unregistered host pointer on older runtimes: treat as host
+    a.type = cudaMemoryTypeUnregistered;
+  }
+  if (a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged) {
+    const int vec4 = ((((uintptr_t)dst) | ((uintptr_t)src)) & 15) == 0;
+    const uint64_t words = bytes / 4;
+    g->launches++;
+    k_copy_words<<<grid_for(vec4 ? words / 4 + 1 : words), 256, 0, s>>>((uint32_t *)dst, (const uint32_t *)src,
+                                                                         words, vec4);
+    return cudaGetLastError();
+  }
+  return cudaMemcpyAsync(dst, src, bytes, cudaMemcpyDefault, s);
+}
+
+// Zero fill by a kernel: cudaMemsetAsync may run on a copy engine and then waits behind a
+// user's large D2H (measured: BFS 1.7 -> 15.7 ms under a concurrent 256 MB D2H).
+__global__ void k_zero_words(uint32_t *__restrict__ dst, uint64_t nwords, int vec4) {
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  const uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x;
+  uint64_t head = 0;
+  if (vec4) {
+    const uint64_t n4 = nwords / 4;
+    for (uint64_t i = i0; i < n4; i += stride) reinterpret_cast<uint4 *>(dst)[i] = make_uint4(0, 0, 0, 0);
+    head = n4 * 4;
+  }
+  for (uint64_t i = head + i0; i < nwords; i += stride) dst[i] = 0u;
+}
+
+cudaError_t fill_zero(gpma *g, void *dst, size_t bytes, cudaStream_t s) {
+  if (!bytes) return cudaSuccess;
+  const uint64_t words = bytes / 4;
+  const int vec4 = (((uintptr_t)dst) & 15) == 0;
+  g->launches++;
+  k_zero_words<<<grid_for(vec4 ? words / 4 + 1 : words), 256, 0, s>>>((uint32_t *)dst, words, vec4);
+  return cudaGetLastError();
+}
+
 int num_sms() {
   static const int v = [] {
     int d = 0, n = 0;
@@ -245,7 +318,7 @@ static void scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) 
   DevBuf &sb = tl_scan ? *tl_scan : g->b_scan;
   ensure(sb, (nt + 1) * sizeof(unsigned long long), s);
   unsigned long long *status = (unsigned long long *)sb.p;
-  cudaMemsetAsync(status, 0, (nt + 1) * sizeof(unsigned long long), s);
+  fill_zero(g, status, (nt + 1) * sizeof(unsigned long long), s);
   GP_LAUNCH(g, k_scan_lookback<T>, (unsigned)nt, SC_THREADS, 0, s, in, out, n, status);
 }
 

@@ -157,7 +157,7 @@ gpma_status query_edges(gpma *g, const uint64_t *keys, uint64_t n, uint32_t *val
   if (!n) return GPMA_OK;
   GP_CHECK(g, ensure(X.stage[0], n * 8, s));
   uint64_t *q = (uint64_t *)X.stage[0].p;
-  GP_CHECK(g, cudaMemcpyAsync(q, keys, n * 8, cudaMemcpyDefault, s));
+  GP_CHECK(g, stage_in(g, q, keys, n * 8, s));
   GP_LAUNCH(g, k_query_edges, grid_for(n), TQ, 0, s, q, n, g->key, g->val, g->head, (uint32_t)(g->cap / g->L),
             g->L, vals, found);
   GP_CHECK(g, cudaGetLastError());
@@ -172,10 +172,10 @@ gpma_status query_neighbors(gpma *g, const uint32_t *verts, uint64_t n, uint64_t
   GP_CHECK(g, ensure(X.lpre, (n + 1) * 8, s));
   uint32_t *vq = (uint32_t *)X.stage[1].p;
   uint64_t *rp = (uint64_t *)X.lpre.p;
-  if (n) GP_CHECK(g, cudaMemcpyAsync(vq, verts, n * 4, cudaMemcpyDefault, s));
+  if (n) GP_CHECK(g, stage_in(g, vq, verts, n * 4, s));
   if (n) GP_LAUNCH(g, k_query_rowsizes, grid_for(n), TQ, 0, s, vq, n, g->deg, g->rb, g->nr, rp);
   scan_u64(g, rp, rp, n, s);
-  GP_CHECK(g, cudaMemcpyAsync(&X.ctrl_h->sum, rp + n, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, readback(g, &X.ctrl_h->sum, rp + n, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   const uint64_t nnz = n ? X.ctrl_h->sum : 0;
   if (nnz_out) *nnz_out = nnz;
@@ -207,15 +207,15 @@ gpma_status query_reachable(gpma *g, const uint32_t *src, const uint32_t *dst, u
   unsigned long long *flags = (unsigned long long *)(qd + 64);   // [0] alive, [1] resolved
   for (uint64_t b0 = 0; b0 < n; b0 += 64) {
     const uint32_t nq = (uint32_t)std::min<uint64_t>(64, n - b0);
-    GP_CHECK(g, cudaMemcpyAsync(qs, src + b0, nq * 4, cudaMemcpyDefault, s));
-    GP_CHECK(g, cudaMemcpyAsync(qd, dst + b0, nq * 4, cudaMemcpyDefault, s));
-    GP_CHECK(g, cudaMemsetAsync(seen, 0, V * 8, s));
-    GP_CHECK(g, cudaMemsetAsync(front, 0, V * 8, s));
-    GP_CHECK(g, cudaMemsetAsync(next, 0, V * 8, s));
+    GP_CHECK(g, stage_in(g, qs, src + b0, nq * 4, s));
+    GP_CHECK(g, stage_in(g, qd, dst + b0, nq * 4, s));
+    GP_CHECK(g, fill_zero(g, seen, V * 8, s));
+    GP_CHECK(g, fill_zero(g, front, V * 8, s));
+    GP_CHECK(g, fill_zero(g, next, V * 8, s));
     GP_LAUNCH(g, k_msbfs_init, 1, 64, 0, s, qs, nq, seen, front);
     const unsigned long long all = nq == 64 ? ~0ull : ((1ull << nq) - 1);
     for (;;) {
-      GP_CHECK(g, cudaMemsetAsync(flags, 0, 16, s));
+      GP_CHECK(g, fill_zero(g, flags, 16, s));
       GP_LAUNCH(g, k_msbfs_answer, 1, 64, 0, s, qd, nq, seen, out + b0, flags + 1);
       GP_LAUNCH(g, k_msbfs_sweep, grid_for(g->cap / 4), TQ, 0, s, g->key, tmask_of(g), g->L, g->cap, front, seen,
                 next);

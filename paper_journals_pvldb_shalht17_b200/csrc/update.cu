@@ -56,6 +56,28 @@ __device__ __forceinline__ uint32_t locate_leaf_rows(const uint64_t *__restrict_
   return lo > a ? lo - 1 : a;
 }
 
+// Slot of key k in leaf `base` (or -1): the occupied prefix of a leaf is sorted and the empty
+// tail is KEY_NONE (> every key), so the scan stops at the first key >= k.  Eight slots are
+// fetched per round with independent 16-B loads (one round trip instead of one per slot).
+__device__ __forceinline__ int find_in_leaf(const uint64_t *__restrict__ key, uint64_t base, uint32_t L,
+                                            uint64_t k) {
+  for (uint32_t p0 = 0; p0 < L; p0 += 8) {
+    ulonglong2 a[4];
+#pragma unroll
+    for (int j = 0; j < 4; ++j)
+      a[j] = p0 + 2 * j < L ? __ldg(reinterpret_cast<const ulonglong2 *>(key + base + p0 + 2 * j))
+                            : make_ulonglong2(KEY_NONE, KEY_NONE);
+#pragma unroll
+    for (int j = 0; j < 4; ++j) {
+      if (a[j].x == k) return (int)(p0 + 2 * j);
+      if (a[j].x > k) return -1;
+      if (a[j].y == k) return (int)(p0 + 2 * j + 1);
+      if (a[j].y > k) return -1;
+    }
+  }
+  return -1;
+}
+
 // ------------------------------------------------------------------ validate
 __global__ void k_validate(const uint64_t *__restrict__ keys, const uint32_t *__restrict__ vals,
                            uint64_t n, uint32_t V, uint32_t rb, uint32_t nr, int check_vals, Ctrl *c) {
@@ -90,12 +112,9 @@ __global__ void k_prepass(const uint64_t *__restrict__ sk, const uint32_t *__res
     if (i + 1 == n || sk[i + 1] != k) {
       uniq = 1;
       t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
-      uint64_t base = (uint64_t)t * L, hit = KEY_NONE;
-      for (uint32_t p = 0; p < L; ++p) {
-        uint64_t x = key[base + p];
-        if (x == k) { hit = base + p; break; }
-        if (x == KEY_NONE || x > k) break;
-      }
+      const uint64_t base = (uint64_t)t * L;
+      const int hp = find_in_leaf(key, base, L, k);
+      const uint64_t hit = hp >= 0 ? base + (uint64_t)hp : KEY_NONE;
       const uint32_t src = (uint32_t)(k >> 32) - rb;   // local row
       const uint32_t bit = hit != KEY_NONE ? 1u << (uint32_t)(hit - base) : 0u;
       if (op == GPMA_INSERT) {
@@ -146,23 +165,18 @@ __global__ void k_lazy_delete(const uint64_t *__restrict__ keys, uint64_t n, con
     const uint64_t k = keys[i];
     const uint32_t t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
     const uint64_t base = (uint64_t)t * L;
-    for (uint32_t p = 0; p < L; ++p) {
-      const uint64_t x = key[base + p];
-      if (x == k) {
-        uint32_t old = val[base + p];
-        while (old != VAL_TOMB) {
-          const uint32_t seen = atomicCAS(&val[base + p], old, VAL_TOMB);
-          if (seen == old) {
-            atomicSub(&cnt[t], 1u);
-            atomicOr(&tmask[t], 1u << p);
-            atomicSub(&deg[(uint32_t)(k >> 32) - rb], 1u);
-            break;
-          }
-          old = seen;
-        }
+    const int p = find_in_leaf(key, base, L, k);
+    if (p < 0) continue;
+    uint32_t old = val[base + p];
+    while (old != VAL_TOMB) {
+      const uint32_t seen = atomicCAS(&val[base + p], old, VAL_TOMB);
+      if (seen == old) {
+        atomicSub(&cnt[t], 1u);
+        atomicOr(&tmask[t], 1u << p);
+        atomicSub(&deg[(uint32_t)(k >> 32) - rb], 1u);
         break;
       }
-      if (x == KEY_NONE || x > k) break;
+      old = seen;
     }
   }
 }
@@ -732,13 +746,13 @@ __global__ void k_raw_counts(const uint64_t *__restrict__ key, const uint32_t *_
 
 // ------------------------------------------------------------------ host driver
 static gpma_status read_ctrl(gpma *g, cudaStream_t s) {
-  GP_CHECK(g, cudaMemcpyAsync(g->ctrl_h, g->ctrl_d, sizeof(Ctrl), cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   return GPMA_OK;
 }
 
 static gpma_status zero_ctrl(gpma *g, cudaStream_t s) {
-  GP_CHECK(g, cudaMemsetAsync(g->ctrl_d, 0, sizeof(Ctrl), s));
+  GP_CHECK(g, fill_zero(g, g->ctrl_d, sizeof(Ctrl), s));
   return GPMA_OK;
 }
 
@@ -798,8 +812,8 @@ gpma_status build_from_sorted(gpma *g, const uint64_t *wk, const uint32_t *wv, u
 }
 
 gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaStream_t s) {
-  GP_CHECK(g, cudaMemcpyAsync(g->key, keys, g->cap * 8, cudaMemcpyDefault, s));
-  GP_CHECK(g, cudaMemcpyAsync(g->val, vals, g->cap * 4, cudaMemcpyDefault, s));
+  GP_CHECK(g, stage_in(g, g->key, keys, g->cap * 8, s));
+  GP_CHECK(g, stage_in(g, g->val, vals, g->cap * 4, s));
   uint64_t nl = g->cap / g->L;
   GP_LAUNCH(g, k_raw_counts, grid_for(nl), TB, 0, s, g->key, g->val, g->cnt, g->row_offset, g->L, nl,
             g->rb, g->nr);
@@ -819,9 +833,9 @@ static gpma_status sort_unique(gpma *g, const uint64_t *keys, const uint32_t *va
   GP_CHECK(g, ensure(g->b_sv[1], n * 4, s));
   uint64_t *k0 = (uint64_t *)g->b_sk[0].p, *k1 = (uint64_t *)g->b_sk[1].p;
   uint32_t *v0 = (uint32_t *)g->b_sv[0].p, *v1 = (uint32_t *)g->b_sv[1].p;
-  GP_CHECK(g, cudaMemcpyAsync(k0, keys, n * 8, cudaMemcpyDefault, s));
-  if (vals) GP_CHECK(g, cudaMemcpyAsync(v0, vals, n * 4, cudaMemcpyDefault, s));
-  else GP_CHECK(g, cudaMemsetAsync(v0, 0, n * 4, s));
+  GP_CHECK(g, stage_in(g, k0, keys, n * 8, s));
+  if (vals) GP_CHECK(g, stage_in(g, v0, vals, n * 4, s));
+  else GP_CHECK(g, fill_zero(g, v0, n * 4, s));
   int sh[8];
   int ns = key_shifts(g->V, sh);
   *which = radix_sort_pairs(g, k0, v0, k1, v1, n, sh, ns, s);
@@ -853,8 +867,8 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
     // stage + validate on device
     GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
     GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
-    GP_CHECK(g, cudaMemcpyAsync(g->b_stage[0].p, keys, n * 8, cudaMemcpyDefault, s));
-    GP_CHECK(g, cudaMemcpyAsync(g->b_stage[1].p, vals, n * 4, cudaMemcpyDefault, s));
+    GP_CHECK(g, stage_in(g, g->b_stage[0].p, keys, n * 8, s));
+    GP_CHECK(g, stage_in(g, g->b_stage[1].p, vals, n * 4, s));
     if ((st = validate(g, (uint64_t *)g->b_stage[0].p, (uint32_t *)g->b_stage[1].p, n, true, s)))
       return st;
     int which;
@@ -870,7 +884,7 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
     GP_LAUNCH(g, k_unique_last, grid_for(n), TB, 0, s, sk, n, keep);
     scan_u32(g, keep, pos, n, s);
     uint32_t mh = 0;
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, pos + n, 4, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, readback(g, &g->ctrl_h->sum, pos + n, 4, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
     mh = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
     m = mh;
@@ -899,7 +913,7 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
   set_geometry(g, cap);
   if ((st = alloc_store(g, cap, &g->key, &g->val, &g->cnt, &g->head, s))) return st;
   GP_CHECK(g, cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s));
-  GP_CHECK(g, cudaMemsetAsync(g->row_offset, 0, ((uint64_t)g->nr + 1) * 8, s));
+  GP_CHECK(g, fill_zero(g, g->row_offset, ((uint64_t)g->nr + 1) * 8, s));
   GP_CHECK(g, cudaMallocAsync((void **)&g->deg, (uint64_t)g->nr * 4 + 4, s));
   if (E > g->tmax[g->h] && !cap_override) {
     g->err = "initial graph exceeds the root bound";
@@ -970,7 +984,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   } else {
     // the single root window, laid out over the whole new array
     uint64_t N;
-    GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, a.nw, 8, cudaMemcpyDeviceToHost, s));
+    GP_CHECK(g, readback(g, &g->ctrl_h->sum, a.nw, 8, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
     N = g->ctrl_h->sum;
     uint64_t nl_new = new_cap / g->L;
@@ -1198,7 +1212,7 @@ static gpma_status double_root(gpma *g, cudaStream_t s) {
   uint64_t *lb = (uint64_t *)g->b_lpre.p;
   GP_LAUNCH(g, k_count_leaf_live, grid_for(nl), TB, 0, s, g->cnt, nl, lb);
   scan_u64(g, lb, lb, nl, s);
-  GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, lb + nl, 8, cudaMemcpyDeviceToHost, s));
+  GP_CHECK(g, readback(g, &g->ctrl_h->sum, lb + nl, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   const uint64_t N = g->ctrl_h->sum;
   GP_CHECK(g, ensure(g->b_wk, std::max<uint64_t>(N, 1) * 8, s));
@@ -1259,7 +1273,7 @@ static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
       GP_LAUNCH(g, k_lock_split, grid_for(nw), TB, 0, s, a.pk, a.pv, a.pt, a.hf, a.widx, nw,
                 (uint64_t *)g->b_pk[cur ^ 1].p, (uint32_t *)g->b_pv[cur ^ 1].p, (uint32_t *)g->b_pt[cur ^ 1].p, ak,
                 av, na);
-      GP_CHECK(g, cudaMemcpyAsync(&g->ctrl_h->sum, a.widx + nw, 4, cudaMemcpyDeviceToHost, s));
+      GP_CHECK(g, readback(g, &g->ctrl_h->sum, a.widx + nw, 4, s));
       GP_CHECK(g, cudaStreamSynchronize(s));
       const uint64_t q = (uint32_t)g->ctrl_h->sum;      // lock winners at this level
       na += nw - q;
@@ -1318,8 +1332,8 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
   uint64_t *ik = (uint64_t *)g->b_stage[0].p;
   uint32_t *iv = (uint32_t *)g->b_stage[1].p;
-  GP_CHECK(g, cudaMemcpyAsync(ik, keys, n * 8, cudaMemcpyDefault, s));
-  if (op == GPMA_INSERT) GP_CHECK(g, cudaMemcpyAsync(iv, vals, n * 4, cudaMemcpyDefault, s));
+  GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));
+  if (op == GPMA_INSERT) GP_CHECK(g, stage_in(g, iv, vals, n * 4, s));
   if ((st = zero_ctrl(g, s))) return st;
   GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, ik, iv, n, g->V, g->rb, g->nr, op == GPMA_INSERT ? 1 : 0,
             g->ctrl_d);
@@ -1352,7 +1366,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   const bool fused = !g->trace_on && !lock;   // the per-level trace needs the generic level-0 step
   if (fused) {
     // level 0 fused: one warp per leaf group, sized by n, counts read on the device
-    GP_CHECK(g, cudaMemsetAsync(keep2, 0, (n + 1) * 4, s));
+    GP_CHECK(g, fill_zero(g, keep2, (n + 1) * 4, s));
     const uint32_t bound = (uint32_t)(op == GPMA_INSERT ? g->tmax[0] : g->tmin[0]);
     GP_LAUNCH(g, k_level0, grid_for((n + 31) / 32 * 32), 256, 0, s, (const uint64_t *)g->b_pk[0].p,
               (const uint32_t *)g->b_pv[0].p, (const uint32_t *)g->b_pt[0].p, pos + n, g->key, g->val, g->cnt,

@@ -15,9 +15,11 @@ from .fanout import AnalyticsFanout
 
 class SlidingWindowPipeline:
     def __init__(self, g, V: int, max_batch: int, nnz_capacity: int, device, rows: int | None = None,
-                 pr_tol: float = 1e-3, concurrent: bool = False, copy_csr: bool = True):
+                 pr_tol: float = 1e-3, concurrent: bool = False, copy_csr: bool = True,
+                 copy_results: bool = True):
         self.g, self.V, self.dev, self.pr_tol = g, V, torch.device(device), pr_tol
         self.copy_csr = copy_csr              # False: the exported CSR stays in HBM (device users)
+        self.copy_results = copy_results      # False: no D2H at all (diagnostics)
         self.fan = AnalyticsFanout(self.dev, priorities=[0, -1, -2, 0]) if concurrent else None
         self.cs = torch.cuda.Stream(self.dev)      # compute
         self.xs = torch.cuda.Stream(self.dev)      # copies
@@ -69,7 +71,9 @@ class SlidingWindowPipeline:
 
             def pr(st):
                 it = g.gpma_pagerank(self.x, warm_start=True, tol_l1=self.pr_tol, stream=st)
-                dx.copy_(self.x, non_blocking=True)
+                # snapshot for the D2H by an SM copy (x * 1.0 is exact), not a D2D cudaMemcpy:
+                # that would queue on a copy engine behind the previous slide's result D2H
+                torch.mul(self.x, 1.0, out=dx)
                 return it
             jobs = [pr, lambda st: g.gpma_cc(lab, stream=st), lambda st: g.gpma_bfs(root, lv, stream=st),
                     lambda st: g.gpma_export_csr(rp, col, cv, stream=st)]
@@ -81,6 +85,9 @@ class SlidingWindowPipeline:
             self.nnz[slot] = r[3]
             self.ev_done[slot].record(s)
         self.xs.wait_event(self.ev_done[slot])
+        if not self.copy_results:
+            self.ev_out[slot].record(self.xs)
+            return
         h = self.h_out[slot]
         n = self.nnz[slot]
         with torch.cuda.stream(self.xs):
