@@ -27,6 +27,7 @@
 #include <cstring>
 
 #include "gpma_internal.cuh"
+#include "sweep.cuh"
 
 namespace gp {
 
@@ -1074,6 +1075,76 @@ __global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ k
   }
 }
 
+// TMA-fed export (sweep.cuh): each stage holds a tile's keys, tombstone masks, values and the
+// output offsets of its leaves (lbase); consumer warps rank the live edges of each 32-slot
+// group with one ballot (a leaf's edges are contiguous in the output from lbase[leaf]) and
+// store (col, val) as coalesced runs, guards setting row_ptr (R8).
+constexpr int EX_T = 1024, EX_S = 3, EX_NC = 4, EX_PER_SM = 4;
+
+struct ExportOp {
+  static constexpr int SIDE = EX_T * 4 + (EX_T / 4) * 8;   // values + lbase of up to T/4 leaves
+  static constexpr int EXTRA = 0;
+  const uint32_t *val;
+  const uint64_t *lbase;
+  uint64_t *row_ptr;
+  uint32_t *col, *cval;
+  uint32_t rb, lgL;
+  __device__ void init(void *) const {}
+  __device__ void finish(void *) const {}
+  __device__ uint32_t side_bytes(uint64_t, uint64_t, uint64_t, uint32_t *m) const {
+    *m = 0;
+    return EX_T * 4 + ((EX_T >> lgL) * 8 + 15) / 16 * 16;
+  }
+  __device__ void side_copy(uint64_t s0, uint32_t, void *dst, uint32_t bytes, uint64_t *bar) const {
+    const uint64_t pol = tma::policy_evict_first();
+    tma::bulk_g2s(dst, val + s0, EX_T * 4, bar, pol);
+    tma::bulk_g2s((unsigned char *)dst + EX_T * 4, lbase + (s0 >> lgL), bytes - EX_T * 4, bar, pol);
+  }
+  template <int G>
+  __device__ __forceinline__ void visit_warp(const uint64_t *sk, const uint32_t *stm, const void *side, uint32_t,
+                                             uint64_t, uint32_t i0, uint32_t L, uint32_t lgL_, void *) const {
+    const uint32_t *sv = (const uint32_t *)side;
+    const uint64_t *lb = (const uint64_t *)((const unsigned char *)side + EX_T * 4);
+    const uint32_t lane = threadIdx.x & 31;
+    const uint32_t below = (1u << lane) - 1u;
+    // lanes of the same leaf inside a 32-slot group (L <= 32, groups are leaf aligned)
+    const uint32_t lmask = L >= 32 ? 0xffffffffu : (((1u << L) - 1u) << (lane & ~(L - 1u)));
+    uint64_t k[G];
+    uint32_t tw[G];
+#pragma unroll
+    for (int j = 0; j < G; ++j) {
+      const uint32_t i = i0 + 32 * j;
+      k[j] = sk[i];
+      tw[j] = stm[i >> lgL_] >> (i & (L - 1));
+    }
+#pragma unroll
+    for (int j = 0; j < G; ++j) {
+      const uint32_t i = i0 + 32 * j;
+      const bool e = live_key(k[j]) && !(tw[j] & 1u);
+      const uint32_t bal = __ballot_sync(0xffffffffu, e);
+      const uint64_t pos = lb[i >> lgL_] + __popc(bal & below & lmask);
+      if (e) {
+        col[pos] = (uint32_t)k[j];
+        cval[pos] = sv[i];
+      } else if (is_guard_key(k[j])) {
+        row_ptr[(k[j] >> 32) - rb + 1] = pos;
+      }
+    }
+  }
+};
+
+__global__ void __launch_bounds__(32 * (EX_NC + 1), 1)
+    k_exp_tma(const uint64_t *__restrict__ key, const uint32_t *__restrict__ tmask, const uint64_t *__restrict__ head,
+              uint64_t cap, uint32_t L, uint32_t lgL, ExportOp op) {
+  sweep_run<EX_T, EX_S, EX_NC>(key, tmask, head, cap, L, lgL, op);
+}
+
+// guard-indexed or not, any store with whole leaf-aligned tiles (GPMA_EXPORT_TMA=0 disables)
+static bool export_use_tma(const gpma *g) {
+  static const int v = [] { const char *e = getenv("GPMA_EXPORT_TMA"); return e ? atoi(e) : 1; }();
+  return v && g->cap >= (uint64_t)EX_T && g->cap % EX_T == 0 && g->L <= 32;
+}
+
 gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val, uint64_t cap_nnz,
                        uint64_t *nnz_out, cudaStream_t s) {
   Scratch &X = g->an[AN_EXPORT];
@@ -1093,8 +1164,20 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
     return GPMA_ERR_INVALID_ARG;
   }
   GP_CHECK(g, fill_zero(g, row_ptr, 8, s));
-  GP_LAUNCH(g, k_exp_write, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, g->val, tmask_of(g), g->L, g->cap, lc,
-            row_ptr, col, val, g->rb);
+  if (export_use_tma(g)) {
+    constexpr size_t sm = sweep_smem<EX_T, EX_S, ExportOp>();
+    static std::atomic<bool> attr{false};
+    if (!attr.load()) {
+      GP_CHECK(g, cudaFuncSetAttribute(k_exp_tma, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm));
+      attr.store(true);
+    }
+    ExportOp op{g->val, lc, row_ptr, col, val, g->rb, ilog2(g->L)};
+    GP_LAUNCH(g, k_exp_tma, num_sms() * EX_PER_SM, 32 * (EX_NC + 1), sm, s, g->key, tmask_of(g), g->head, g->cap,
+              g->L, ilog2(g->L), op);
+  } else {
+    GP_LAUNCH(g, k_exp_write, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, g->val, tmask_of(g), g->L,
+              g->cap, lc, row_ptr, col, val, g->rb);
+  }
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }

@@ -117,9 +117,9 @@ __device__ __forceinline__ TileRows tile_rows(uint64_t h_lo, uint64_t h_hi, uint
 
 // The generic persistent sweep.  Op must provide
 //   static constexpr int SIDE;                       side bytes per stage (multiple of 16)
-//   __device__ uint32_t side_bytes(uint64_t h_lo, uint64_t h_hi, uint32_t *meta) const;
+//   __device__ uint32_t side_bytes(uint64_t s0, uint64_t h_lo, uint64_t h_hi, uint32_t *meta) const;
 //       producer lane: bytes of the tile's side slice (0 = none) and a word for the consumers
-//   __device__ void side_copy(uint32_t meta, void *dst, uint32_t bytes, uint64_t *bar) const;
+//   __device__ void side_copy(uint64_t s0, uint32_t meta, void *dst, uint32_t bytes, uint64_t *bar) const;
 //       producer lane: issue the side copies (completing on bar)
 //   template <int G> __device__ void visit_warp(const uint64_t *key, const uint32_t *tm,
 //                         const void *side, uint32_t meta, uint64_t s0, uint32_t i0, uint32_t L,
@@ -192,12 +192,12 @@ __device__ __forceinline__ void sweep_run(const uint64_t *__restrict__ key, cons
           uint32_t m = 0;
           // expected bytes first (the copies may complete before the arrive otherwise)
           const uint32_t kb = T * 8, tb = (lpt * 4 + 15) & ~15u;
-          uint32_t sb = op.side_bytes(h_lo, h_hi, &m);
+          uint32_t sb = op.side_bytes(s0, h_lo, h_hi, &m);
           meta[s] = m;
           tma::mbar_arrive_tx(&full[s], kb + tb + sb);
           tma::bulk_g2s(st[s].key, key + s0, kb, &full[s], pol);
           tma::bulk_g2s(st[s].tm, tmask + (s0 >> lgL), tb, &full[s], pol);
-          if (sb) op.side_copy(m, st[s].side, sb, &full[s]);
+          if (sb) op.side_copy(s0, m, st[s].side, sb, &full[s]);
         }
       }
       hcur = hnext;
