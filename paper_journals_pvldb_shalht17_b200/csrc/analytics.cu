@@ -45,7 +45,7 @@ __device__ __forceinline__ void load4(const uint64_t *__restrict__ key, const ui
   ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(key + s4));
   ulonglong2 b = __ldcs(reinterpret_cast<const ulonglong2 *>(key + s4 + 2));
   o.k[0] = a.x; o.k[1] = a.y; o.k[2] = b.x; o.k[3] = b.y;
-  o.tb = (__ldg(tmask + s4 / L) >> (uint32_t)(s4 % L)) & 0xFu;
+  o.tb = (__ldg(tmask + leaf_div(s4, L)) >> leaf_mod(s4, L)) & 0xFu;
 }
 
 __device__ __forceinline__ uint64_t l2_evict_last_policy() {
@@ -62,7 +62,7 @@ __device__ __forceinline__ bool edge_at(const uint64_t *__restrict__ key, const 
   uint64_t x = __ldcs(key + s);
   *k = x;
   if (!live_key(x)) return false;
-  return !((__ldg(tmask + s / L) >> (uint32_t)(s % L)) & 1u);
+  return !((__ldg(tmask + leaf_div(s, L)) >> leaf_mod(s, L)) & 1u);
 }
 
 __device__ __forceinline__ uint32_t upper_bound_u64(const uint64_t *__restrict__ a, uint32_t lo, uint32_t hi,
@@ -493,7 +493,7 @@ __global__ void __launch_bounds__(TA) k_cc_sample(const uint64_t *__restrict__ k
       const uint64_t s = t * 4 + j;
       const uint64_t pk = j ? sl.k[j - 1] : prev;
       if (!edge4(sl, j)) continue;
-      const bool first = (s % L == 0) || pk == KEY_NONE || (pk >> 32) != (sl.k[j] >> 32);
+      const bool first = (leaf_mod(s, L) == 0) || pk == KEY_NONE || (pk >> 32) != (sl.k[j] >> 32);
       if (!first) continue;
       uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
       if (u != v && cc_ld<H>(p + u, pol) != cc_ld<H>(p + v, pol)) cc_hook<H>(p, u, v, pol);
@@ -521,7 +521,7 @@ __global__ void __launch_bounds__(TA) k_cc_sample_rows(const uint64_t *__restric
         sl |= (uint64_t)(L - 1);
         continue;
       }
-      if ((__ldg(tmask + sl / L) >> (uint32_t)(sl % L)) & 1u) continue;   // tombstone
+      if ((__ldg(tmask + leaf_div(sl, L)) >> leaf_mod(sl, L)) & 1u) continue;   // tombstone
       const uint32_t v = (uint32_t)k;
       ++found;
       if (u != v && cc_ld<H>(p + u, pol) != cc_ld<H>(p + v, pol)) cc_hook<H>(p, u, v, pol);
@@ -783,7 +783,7 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
   const uint64_t chunk = (((cap + nwarps - 1) / nwarps) + 32 * U - 1) / (32 * U) * (32 * U);
   const uint64_t beg = w * chunk, end = min(beg + chunk, cap);
   if (beg >= end) return;
-  const uint64_t h0 = head[beg / L];
+  const uint64_t h0 = head[leaf_div(beg, L)];
   if (h0 == KEY_NONE) return;                            // no key at or after this chunk
   uint32_t ub = (uint32_t)(h0 >> 32) - rb;               // lower bound of the chunk's rows
   A win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
@@ -794,7 +794,7 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
     for (int j = 0; j < U; ++j) {
       const uint64_t s = base + j * 32 + lane;
       kk[j] = s < end ? __ldcs(key + s) : KEY_NONE;
-      tt[j] = s < end ? (__ldg(tmask + s / L) >> (uint32_t)(s % L)) & 1u : 1u;
+      tt[j] = s < end ? (__ldg(tmask + leaf_div(s, L)) >> leaf_mod(s, L)) & 1u : 1u;
     }
   };
   fetch(beg, k, tb);
@@ -1051,7 +1051,7 @@ __global__ void __launch_bounds__(TA) k_exp_write(const uint64_t *__restrict__ k
     }
     const uint32_t total = __shfl_sync(0xffffffffu, incl, 31);
     const uint64_t t0 = t - lane;                               // warp's first slot group
-    const uint64_t wbase = t0 < n4 ? lbase[(t0 * 4) / L] : 0;
+    const uint64_t wbase = t0 < n4 ? lbase[leaf_div(t0 * 4, L)] : 0;
     uint4 vv = make_uint4(0, 0, 0, 0);
     if (e) vv = __ldcs(reinterpret_cast<const uint4 *>(val + t * 4));
     const uint32_t vs[4] = {vv.x, vv.y, vv.z, vv.w};

@@ -22,6 +22,17 @@ constexpr int MAX_RESIDENT_BLOCKS = 148 * 8;  // grid-stride kernels: 8 x 256-th
 // the skewed (RMAT) work per chunk balances out -- measured 10-20% faster than one wave.
 constexpr int SWEEP_BLOCKS = 148 * 64;
 
+// L (slots per leaf) is a power of two (R3; gpma_create / gpma_create_raw reject others):
+// slot -> leaf and slot-in-leaf are a shift and a mask, not a 64-bit division by a runtime L
+__host__ __device__ __forceinline__ uint64_t leaf_div(uint64_t s, uint32_t L) {
+#ifdef __CUDA_ARCH__
+  return s >> (__ffs(L) - 1);
+#else
+  return s >> __builtin_ctz(L);
+#endif
+}
+__host__ __device__ __forceinline__ uint32_t leaf_mod(uint64_t s, uint32_t L) { return (uint32_t)s & (L - 1); }
+
 __host__ __device__ inline bool is_guard_key(uint64_t k) {
   return k != KEY_NONE && (uint32_t)k == COL_GUARD;
 }

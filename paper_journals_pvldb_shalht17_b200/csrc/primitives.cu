@@ -51,7 +51,15 @@ long prof_begin(gpma *g, const char *name, cudaStream_t s) {
     // exact match on the kernel name without template arguments
     const char *lt = strchr(name, '<');
     size_t n = lt ? (size_t)(lt - name) : strlen(name);
-    if (g->prof_filter.size() != n || strncmp(g->prof_filter.c_str(), name, n) != 0) return -1;
+    // (a comma-separated filter matches any of its names)
+    bool hit = false;
+    for (size_t a = 0; a <= g->prof_filter.size() && !hit;) {
+      size_t b = g->prof_filter.find(',', a);
+      if (b == std::string::npos) b = g->prof_filter.size();
+      hit = (b - a == n) && strncmp(g->prof_filter.c_str() + a, name, n) == 0;
+      a = b + 1;
+    }
+    if (!hit) return -1;
   }
   std::lock_guard<std::mutex> lk(g->mu);
   size_t e0 = take_event(g), e1 = take_event(g);

@@ -79,7 +79,7 @@ __global__ void k_query_rows(const uint32_t *__restrict__ verts, uint64_t n, con
       uint64_t k = KEY_NONE;
       if (s < b) {
         k = key[s];
-        e = k != KEY_NONE && (uint32_t)k != COL_GUARD && !((tmask[s / L] >> (uint32_t)(s % L)) & 1u);
+        e = k != KEY_NONE && (uint32_t)k != COL_GUARD && !((tmask[leaf_div(s, L)] >> leaf_mod(s, L)) & 1u);
       }
       const uint32_t bal = __ballot_sync(0xffffffffu, e);
       if (e) {
@@ -112,7 +112,7 @@ __global__ void __launch_bounds__(TQ) k_msbfs_sweep(const uint64_t *__restrict__
     const ulonglong2 ka = __ldcs(reinterpret_cast<const ulonglong2 *>(key + s4));
     const ulonglong2 kb = __ldcs(reinterpret_cast<const ulonglong2 *>(key + s4 + 2));
     const uint64_t k[4] = {ka.x, ka.y, kb.x, kb.y};
-    const uint32_t tb = (__ldg(tmask + s4 / L) >> (uint32_t)(s4 % L)) & 0xFu;
+    const uint32_t tb = (__ldg(tmask + leaf_div(s4, L)) >> leaf_mod(s4, L)) & 0xFu;
 #pragma unroll
     for (int j = 0; j < 4; ++j) {
       if (k[j] == KEY_NONE || (uint32_t)k[j] == COL_GUARD || ((tb >> j) & 1u)) continue;

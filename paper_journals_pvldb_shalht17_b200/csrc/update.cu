@@ -46,8 +46,8 @@ __device__ __forceinline__ uint32_t locate_leaf_rows(const uint64_t *__restrict_
   if (!ro) return locate_leaf(head, nleaves, k);
   const uint32_t u = (uint32_t)(k >> 32) - rb;
   const ulonglong2 r = make_ulonglong2(__ldg(ro + u), __ldg(ro + u + 1));
-  const uint32_t a = (uint32_t)(r.x / L);
-  uint32_t lo = a, hi = min((uint32_t)(r.y / L) + 1, nleaves);
+  const uint32_t a = (uint32_t)leaf_div(r.x, L);
+  uint32_t lo = a, hi = min((uint32_t)leaf_div(r.y, L) + 1, nleaves);
   while (lo < hi) {
     uint32_t mid = (lo + hi) >> 1;
     if (__ldg(head + mid) <= k) lo = mid + 1;
@@ -588,7 +588,7 @@ __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *_
   const uint64_t cap = nleaves * L;
   for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
        s += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t l = s / L, p = s % L;
+    uint64_t l = leaf_div(s, L), p = leaf_mod(s, L);
     uint64_t lo = l * N / nleaves, hi = (l + 1) * N / nleaves;
     if (p < hi - lo) {
       uint64_t k = wk[lo + p];
@@ -1196,7 +1196,7 @@ __global__ void k_gather_live(const uint64_t *__restrict__ key, const uint32_t *
     const bool live = s < cap && k != KEY_NONE && v != VAL_TOMB;
     const uint32_t bal = __ballot_sync(0xffffffffu, live);
     if (live) {
-      const uint64_t d = lbase[s / L] + __popc(bal & leafmask & lt);
+      const uint64_t d = lbase[leaf_div(s, L)] + __popc(bal & leafmask & lt);
       wk[d] = k;
       wv[d] = v;
     }
