@@ -306,7 +306,7 @@ __global__ void __launch_bounds__(TA) k_bfs_sweep(const uint64_t *__restrict__ k
   for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4;
        t += (uint64_t)gridDim.x * blockDim.x) {
     Slot4 sl;
-    load4(key, tmask, L, (uint64_t)alist[t / tpl] * L + (t % tpl) * 4, sl);
+    load4(key, tmask, L, (uint64_t)alist[leaf_div(t, tpl)] * L + leaf_mod(t, tpl) * 4, sl);   // tpl = L/4: a power of two
 #pragma unroll
     for (int j = 0; j < 4; ++j) {
       if (!edge4(sl, j)) continue;
@@ -320,8 +320,8 @@ __global__ void __launch_bounds__(TA) k_bfs_sweep(const uint64_t *__restrict__ k
 
 // frontiers up to this size use row expansion (GPMA_BFS_SPARSE overrides)
 static uint32_t bfs_sparse_f() {
-  static const uint32_t v = [] { const char *e = getenv("GPMA_BFS_SPARSE"); return e ? (uint32_t)atol(e) : 32768u; }();
-  return v;
+  const char *e = getenv("GPMA_BFS_SPARSE");              // read per call: tests switch it
+  return e ? (uint32_t)atol(e) : 32768u;
 }
 
 gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
