@@ -582,8 +582,8 @@ static int cc_hint() {
 // sampled first round: row based when every row has its guard (GPMA_CC_SAMPLE=0 forces the
 // slot sweep), else the (source, leaf)-run sweep
 static int cc_sample_mode() {
-  static const int v = [] { const char *e = getenv("GPMA_CC_SAMPLE"); return e ? atoi(e) : 2; }();
-  return v;
+  const char *e = getenv("GPMA_CC_SAMPLE");               // read per call: tests switch it
+  return e ? atoi(e) : 2;
 }
 
 static cudaError_t cc_sample(gpma *g, uint32_t *p, cudaStream_t s) {

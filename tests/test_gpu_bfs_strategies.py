@@ -64,3 +64,16 @@ def test_bfs_every_strategy(scale):
             with env(GPMA_BFS_SPARSE=sparse):
                 got = gpu_bfs(g, root)
             assert np.array_equal(got, want), f"root {root} sparse {sparse}"
+
+
+@pytest.mark.parametrize("scale", [10, 16])
+def test_cc_every_sample_strategy(scale):
+    """CC (Soman et al.; R19 weak components, min-id labels) with every first-round
+    sample: slot sweep (0), first one / two edges per row (1, 2)."""
+    sw, g, o = _store(scale)
+    want = o.cc()
+    from tests.gpu_helpers import gpu_cc
+    for mode in ("0", "1", "2"):
+        with env(GPMA_CC_SAMPLE=mode):
+            got = gpu_cc(g)
+        assert np.array_equal(got, want), f"sample mode {mode}"
