@@ -278,6 +278,7 @@ def run_gpma(args, rank, world, lrank):
                     if j + 1 <= args.e2e_steps:
                         pipe.stage((j + 1) % 2, *batches[j + 1])
                     pipe.run(j % 2, roots[j])
+                pipe.flush()                               # the last slide's result D2H
                 e1.record(pipe.xs)
                 pipe.drain()
                 wall = time.perf_counter() - t0e
