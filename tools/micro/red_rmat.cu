@@ -49,6 +49,19 @@ __global__ void k_gen_only(unsigned long long *y, uint64_t n_ops, int scale, int
     acc ^= mode ? rmat_dst(i, scale) : (uint32_t)(mix(i) & (V - 1));
   if (acc == 0x12345678) y[0] = acc;
 }
+// REDs with the destinations in a hot bitmap skipped (what a shared-memory aggregation of the
+// hot destinations would leave to L2): measures the same-address serialisation on hot lines
+__global__ void k_red_buf_skip(unsigned long long *y, const uint32_t *dst, uint64_t n_ops, const uint32_t *hot) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n_ops; i += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t d = __ldcs(dst + i);
+    if ((__ldg(hot + (d >> 5)) >> (d & 31)) & 1u) continue;
+    atomicAdd(&y[d], 1ull);
+  }
+}
+__global__ void k_mark_hot(const unsigned long long *cnt, uint32_t V, unsigned long long thr, uint32_t *hot) {
+  for (uint32_t v = blockIdx.x * blockDim.x + threadIdx.x; v < V; v += gridDim.x * blockDim.x)
+    if (cnt[v] >= thr) atomicOr(hot + (v >> 5), 1u << (v & 31));
+}
 int main() {
   const uint64_t ops = 134217728;
   const int scale = 24;
@@ -112,6 +125,26 @@ int main() {
         ++top; acc += c;
         if (top == marks[mi]) { printf("top %llu vertices: %.1f%% of REDs (min count %lld)\n", top, 100.0 * acc / ops, (long long)c); ++mi; }
       }
+    }
+  }
+  {
+    unsigned long long *cnt;
+    cudaMalloc(&cnt, 8ull << scale);
+    cudaMemset(cnt, 0, 8ull << scale);
+    k_red_buf<<<148 * 8, 256>>>(cnt, dst, ops, 1u << 24);   // rmat dst (last generated mode)
+    uint32_t *hot;
+    cudaMalloc(&hot, (1u << scale) / 8);
+    for (unsigned long long thr : {~0ull, 58449ull, 18328ull, 5853ull, 1882ull, 615ull}) {
+      cudaMemset(hot, 0, (1u << scale) / 8);
+      k_mark_hot<<<148 * 8, 256>>>(cnt, 1u << scale, thr, hot);
+      float ms;
+      k_red_buf_skip<<<148 * 8, 256>>>(y, dst, ops, hot);
+      cudaEventRecord(a);
+      k_red_buf_skip<<<148 * 8, 256>>>(y, dst, ops, hot);
+      cudaEventRecord(b);
+      cudaEventSynchronize(b);
+      cudaEventElapsedTime(&ms, a, b);
+      printf("rmat REDs, destinations with count >= %llu skipped: %.3f ms\n", thr, ms);
     }
   }
   return 0;
