@@ -172,6 +172,8 @@ void free_handle(gpma *g) {
   if (g->row_offset) cudaFreeAsync(g->row_offset, s);
   if (g->deg) cudaFreeAsync(g->deg, s);
   cudaStreamSynchronize(s);
+  for (gp::UpdGraph &u : g->ugraph)
+    if (u.exec) cudaGraphExecDestroy(u.exec);
   for (cudaEvent_t e : g->ev_pool) cudaEventDestroy(e);
   if (g->ctrl_d) cudaFree(g->ctrl_d);
   if (g->ctrl_h) cudaFreeHost(g->ctrl_h);

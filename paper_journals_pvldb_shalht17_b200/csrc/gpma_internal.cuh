@@ -78,6 +78,18 @@ struct Scratch {
   Ctrl *ctrl_h = nullptr;         // pinned mirror
 };
 
+// Replayable prefix of one update batch (everything up to its single host read-back) as a
+// CUDA graph: small batches are bound by host launch overhead (~12 launches per insert), a
+// graph replays them with one launch.  Valid while the signature -- batch shape plus every
+// pointer / scalar the prefix bakes into its kernels -- is unchanged.
+struct UpdGraph {
+  std::vector<uint64_t> sig;      // signature of the captured graph
+  std::vector<uint64_t> seen;     // signature after the last un-captured run of this op
+  cudaGraphExec_t exec = nullptr;
+  uint64_t nlaunch = 0;           // kernels in the graph (launch accounting)
+  int which = 0;                  // sort result buffer of the captured shape
+};
+
 }  // namespace gp
 
 struct gpma {
@@ -86,6 +98,8 @@ struct gpma {
   uint32_t rb = 0, nr = 0;        // owned rows [rb, rb + nr) (shard, R24); nr = V unsharded
   uint32_t algorithm = 0;         // 0 = GPMA+ (Alg. 4), 1 = GPMA lock-based (Alg. 1)
   bool rows_indexed = false;      // every owned row has its guard: row_offset locates leaves
+  gp::UpdGraph ugraph[2];         // per op (insert, delete)
+  bool graphs_off = false;        // a capture failed once: plain launches from then on
   uint64_t cap = 0;
   uint32_t rho0 = 800, rhoh = 4000, tau0 = 9200, tauh = 8000, init_bp = 6000;
   std::vector<uint64_t> tmin, tmax;

@@ -1318,22 +1318,12 @@ static gpma_status status_of(gpma *g) {
   return GPMA_OK;
 }
 
-// One batch.  Validation runs on the device and every mutating kernel bails out when it
-// flagged the batch, so the common insert path (sort -> pre-pass -> fused level 0) needs a
-// single host round trip; the generic levels >= 1 and the resize follow only when level 0
-// leaves updates pending.
-gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op,
-                         cudaStream_t s) {
+// The prefix of one batch, up to and including the read-back of the control block (no host
+// synchronisation inside): validate, then lazy delete, or sort -> pre-pass -> compact ->
+// fused level 0 -> summary.  *which = the sort's result buffer.
+static gpma_status upd_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int *which,
+                              cudaStream_t s) {
   gpma_status st;
-  g->last = gpma_stats_t{};
-  g->trace.clear();
-  if (n == 0) return GPMA_OK;
-  GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
-  GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
-  uint64_t *ik = (uint64_t *)g->b_stage[0].p;
-  uint32_t *iv = (uint32_t *)g->b_stage[1].p;
-  GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));
-  if (op == GPMA_INSERT) GP_CHECK(g, stage_in(g, iv, vals, n * 4, s));
   if ((st = zero_ctrl(g, s))) return st;
   GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, ik, iv, n, g->V, g->rb, g->nr, op == GPMA_INSERT ? 1 : 0,
             g->ctrl_d);
@@ -1341,15 +1331,13 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
     GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
               tmask_of(g), g->deg, g->rb, g->ctrl_d, g->rows_indexed ? g->row_offset : nullptr);
-    if ((st = read_ctrl(g, s))) return st;
-    g->last.last_unique = n;   // not deduplicated: lazy deletes are idempotent
-    return status_of(g);
+    GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
+    return GPMA_OK;
   }
-  int which;
   uint64_t m;
-  if ((st = sort_unique(g, ik, op == GPMA_INSERT ? iv : nullptr, n, &m, false, &which, s))) return st;
-  const uint64_t *sk = (const uint64_t *)g->b_sk[which].p;
-  const uint32_t *sv = (const uint32_t *)g->b_sv[which].p;
+  if ((st = sort_unique(g, ik, op == GPMA_INSERT ? iv : nullptr, n, &m, false, which, s))) return st;
+  const uint64_t *sk = (const uint64_t *)g->b_sk[*which].p;
+  const uint32_t *sv = (const uint32_t *)g->b_sv[*which].p;
   GP_CHECK(g, ensure(g->b_keep, (n + 1) * 4, s));
   GP_CHECK(g, ensure(g->b_pos, (n + 1) * 4, s));
   GP_CHECK(g, ensure(g->b_tgt, (n + 1) * 4, s));
@@ -1375,7 +1363,110 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
     scan_u32(g, keep2, kpos, n, s);
   }
   GP_LAUNCH(g, k_upd_summary, 1, 1, 0, s, pos, fused ? kpos : nullptr, n, g->ctrl_d);
-  if ((st = read_ctrl(g, s))) return st;             // the one host round trip of the batch
+  GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
+  return GPMA_OK;
+}
+
+// everything the prefix bakes into its launches
+static std::vector<uint64_t> upd_signature(gpma *g, uint64_t n, int op) {
+  std::vector<uint64_t> v = {n, (uint64_t)op, g->mode, g->algorithm, g->V, g->rb, g->nr, g->cap, g->L, g->h,
+                             g->tmax.empty() ? 0 : g->tmax[0], g->tmin.empty() ? 0 : g->tmin[0],
+                             (uint64_t)g->rows_indexed, (uint64_t)g->trace_on,
+                             (uint64_t)(uintptr_t)g->key, (uint64_t)(uintptr_t)g->val, (uint64_t)(uintptr_t)g->cnt,
+                             (uint64_t)(uintptr_t)g->deg, (uint64_t)(uintptr_t)g->head,
+                             (uint64_t)(uintptr_t)g->row_offset, (uint64_t)(uintptr_t)g->ctrl_d,
+                             (uint64_t)(uintptr_t)g->ctrl_h, (uint64_t)(uintptr_t)tl_scan};
+  const DevBuf *bufs[] = {&g->b_sk[0], &g->b_sk[1], &g->b_sv[0], &g->b_sv[1], &g->b_keep, &g->b_pos, &g->b_tgt,
+                          &g->b_pk[0], &g->b_pk[1], &g->b_pv[0], &g->b_pv[1], &g->b_pt[0], &g->b_pt[1],
+                          &g->b_hf, &g->b_widx, &g->b_wfirst, &g->b_acc, &g->b_aidx, &g->b_alist, &g->b_nw,
+                          &g->b_woff, &g->b_keep2, &g->b_kpos, &g->b_lpre, &g->b_wk, &g->b_wv, &g->b_dirty,
+                          &g->b_scan, &g->b_hist, &g->b_stage[0], &g->b_stage[1], &g->b_stage[2],
+                          &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3};
+  for (const DevBuf *b : bufs) {
+    v.push_back((uint64_t)(uintptr_t)b->p);
+    v.push_back(b->bytes);
+  }
+  return v;
+}
+
+// GPMA_UPD_GRAPH=0 disables graph replay (read per call)
+static bool upd_graph_on(gpma *g) {
+  if (g->graphs_off || g->trace_on || !g->prof_filter.empty()) return false;
+  const char *e = getenv("GPMA_UPD_GRAPH");
+  return !e || atoi(e) != 0;
+}
+
+// Run the prefix: replay the cached graph when the signature matches; capture it on the second
+// run of an unchanged shape (the first run sized every buffer, so the capture allocates
+// nothing); plain launches otherwise.
+static gpma_status run_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int *which,
+                              cudaStream_t s) {
+  if (!s || !upd_graph_on(g)) return upd_prefix(g, ik, iv, n, op, which, s);   // (no capture on the legacy stream)
+  UpdGraph &G = g->ugraph[op == GPMA_INSERT ? 0 : 1];
+  std::vector<uint64_t> sig = upd_signature(g, n, op);
+  if (G.exec && G.sig == sig) {
+    GP_CHECK(g, cudaGraphLaunch(G.exec, s));
+    g->launches += G.nlaunch;
+    *which = G.which;
+    return GPMA_OK;
+  }
+  if (G.seen != sig) {
+    gpma_status st = upd_prefix(g, ik, iv, n, op, which, s);
+    G.seen = upd_signature(g, n, op);
+    return st;
+  }
+  cudaGraph_t graph = nullptr;
+  const uint64_t l0 = g->launches;
+  GP_CHECK(g, cudaStreamBeginCapture(s, cudaStreamCaptureModeRelaxed));
+  gpma_status st = upd_prefix(g, ik, iv, n, op, which, s);
+  cudaError_t e = cudaStreamEndCapture(s, &graph);
+  if (st) return st;
+  cudaGraphExec_t exec = nullptr;
+  if (e == cudaSuccess && upd_signature(g, n, op) == sig) e = cudaGraphInstantiate(&exec, graph, 0);
+  else if (e == cudaSuccess) e = cudaErrorNotSupported;   // the capture allocated: never replay it
+  if (graph) cudaGraphDestroy(graph);
+  if (e != cudaSuccess) {                 // fall back for good; run the prefix plainly now
+    cudaGetLastError();
+    g->graphs_off = true;
+    g->launches = l0;
+    return upd_prefix(g, ik, iv, n, op, which, s);
+  }
+  if (G.exec) cudaGraphExecDestroy(G.exec);
+  G.exec = exec;
+  G.sig = sig;
+  G.nlaunch = g->launches - l0;
+  G.which = *which;
+  GP_CHECK(g, cudaGraphLaunch(exec, s));
+  return GPMA_OK;
+}
+
+// One batch.  Validation runs on the device and every mutating kernel bails out when it
+// flagged the batch, so the common insert path (sort -> pre-pass -> fused level 0) needs a
+// single host round trip; the generic levels >= 1 and the resize follow only when level 0
+// leaves updates pending.
+gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op,
+                         cudaStream_t s) {
+  gpma_status st;
+  g->last = gpma_stats_t{};
+  g->trace.clear();
+  if (n == 0) return GPMA_OK;
+  GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
+  GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
+  uint64_t *ik = (uint64_t *)g->b_stage[0].p;
+  uint32_t *iv = (uint32_t *)g->b_stage[1].p;
+  GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));
+  if (op == GPMA_INSERT) GP_CHECK(g, stage_in(g, iv, vals, n * 4, s));
+  const uint64_t nl = g->cap / g->L;
+  int which = 0;
+  if ((st = run_prefix(g, ik, iv, n, op, &which, s))) return st;
+  GP_CHECK(g, cudaStreamSynchronize(s));             // the one host round trip of the batch
+  if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
+    g->last.last_unique = n;   // not deduplicated: lazy deletes are idempotent
+    return status_of(g);
+  }
+  uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
+  const bool lock = op == GPMA_INSERT && g->algorithm == 1;   // GPMA (Alg. 1) instead of GPMA+
+  const bool fused = !g->trace_on && !lock;
   if ((st = status_of(g))) return st;
   uint64_t p = (uint32_t)g->ctrl_h->sum;
   g->last.last_unique = g->ctrl_h->nunique;
