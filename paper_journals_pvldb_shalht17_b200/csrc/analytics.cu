@@ -261,9 +261,16 @@ __global__ void __launch_bounds__(TA) k_bfs_leaf_active(const uint64_t *__restri
       act[k] = 0;
       if (h0[k] != KEY_NONE) {
         const uint32_t ua = (uint32_t)(h0[k] >> 32);
-        const uint32_t ub = h1[k] == KEY_NONE ? V - 1 : (uint32_t)(h1[k] >> 32);
-        for (uint32_t u = ua; u <= ub && u < V; ++u)
-          if ((__ldg(bm + (u >> 5)) >> (u & 31)) & 1u) { act[k] = 1; break; }
+        const uint32_t ub = min(h1[k] == KEY_NONE ? V - 1 : (uint32_t)(h1[k] >> 32), V - 1);
+        // frontier bits of sources [ua, ub], a word at a time (one or two words when every
+        // row has its guard: a leaf spans at most L + 1 sources)
+        const uint32_t w0 = ua >> 5, w1 = ub >> 5;
+        for (uint32_t w = w0; w <= w1 && ua <= ub; ++w) {
+          uint32_t m = __ldg(bm + w);
+          if (w == w0) m &= ~0u << (ua & 31);
+          if (w == w1 && (ub & 31) != 31) m &= (2u << (ub & 31)) - 1u;
+          if (m) { act[k] = 1; break; }
+        }
       }
       bal[k] = __ballot_sync(0xffffffffu, act[k]);
       if (lane == 0) wofs[k * (TA / 32) + warp] = __popc(bal[k]);
