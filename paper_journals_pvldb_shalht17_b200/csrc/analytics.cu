@@ -536,15 +536,45 @@ __global__ void __launch_bounds__(TA) k_cc_sample_rows(const uint64_t *__restric
   }
 }
 
-__global__ void k_cc_compress(uint32_t *p, uint32_t V) {
-  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
-       v += (uint64_t)gridDim.x * blockDim.x) {
-    volatile uint32_t *vp = p;
-    uint32_t x = vp[v], nx;
-    while ((nx = vp[x]) != x) x = nx;
-    vp[v] = x;
+// Root of every vertex, CC_ILP vertices per thread chased in lockstep.  Chain steps load
+// through L1 (ld.global.ca): almost every chain ends on the giant component's root, and one L2
+// word read by every warp serialised the pass on its slice.  A stale L1 value is still an
+// ancestor (compression only moves parents toward the root, roots never change here), so
+// every chain still ends on its root.  out == p: full compression in place; else out[v] = root.
+constexpr int CC_ILP = 4;
+__device__ __forceinline__ void cc_roots(uint32_t *p, uint32_t *out, uint32_t V) {
+  volatile uint32_t *vp = p;
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t v0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v0 < V; v0 += CC_ILP * stride) {
+    uint32_t x[CC_ILP];
+    uint32_t live = 0;                                     // bit j: chain j not at its root yet
+#pragma unroll
+    for (int j = 0; j < CC_ILP; ++j) {
+      const uint64_t v = v0 + j * stride;
+      x[j] = v < V ? vp[v] : 0u;
+      if (v < V) live |= 1u << j;
+    }
+    while (live) {
+#pragma unroll
+      for (int j = 0; j < CC_ILP; ++j) {
+        if (!((live >> j) & 1u)) continue;
+        const uint32_t nx = __ldca(p + x[j]);
+        if (nx == x[j]) live &= ~(1u << j);
+        else x[j] = nx;
+      }
+    }
+#pragma unroll
+    for (int j = 0; j < CC_ILP; ++j) {
+      const uint64_t v = v0 + j * stride;
+      if (v < V) {
+        if (out == p) vp[v] = x[j];
+        else out[v] = x[j];
+      }
+    }
   }
 }
+
+__global__ void k_cc_compress(uint32_t *p, uint32_t V) { cc_roots(p, p, V); }
 
 template <bool H>
 __device__ __forceinline__ void cc_group(const Slot4 &sl, uint32_t *p, uint64_t pol) {
@@ -609,15 +639,7 @@ static cudaError_t cc_sample(gpma *g, uint32_t *p, cudaStream_t s) {
   return cudaGetLastError();
 }
 
-__global__ void k_cc_final(uint32_t *p, uint32_t *labels, uint32_t V) {
-  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V;
-       v += (uint64_t)gridDim.x * blockDim.x) {
-    volatile uint32_t *vp = p;
-    uint32_t x = (uint32_t)v, nx;
-    while ((nx = vp[x]) != x) x = nx;
-    labels[v] = x;
-  }
-}
+__global__ void k_cc_final(uint32_t *p, uint32_t *labels, uint32_t V) { cc_roots(p, labels, V); }
 
 __global__ void k_cc_changed(const uint32_t *__restrict__ a, const uint32_t *__restrict__ b, uint32_t V, Ctrl *c) {
   uint64_t n = 0;
