@@ -437,13 +437,16 @@ __device__ __forceinline__ uint32_t cc_cas(uint32_t *a, uint32_t cmp, uint32_t v
   return atomicCAS(a, cmp, v);                 // (atom.cas takes no L2 cache hint on sm_100a)
 }
 
-template <bool H>
+// F: chain steps through L1 (a stale parent is still an ancestor; the CAS in cc_hook checks
+// rootness against L2), so a giant component's root word is not re-read from one L2 slice by
+// every chain
+template <bool H, bool F = false>
 __device__ __forceinline__ uint32_t cc_find(uint32_t *p, uint32_t x, uint64_t pol) {
   // path halving on a forest with parent[x] <= x (roots are the minima)
   uint32_t cur = cc_ld<H>(p + x, pol);
   if (cur != x) {
     uint32_t prev = x, next;
-    while (cur > (next = cc_ld<H>(p + cur, pol))) {
+    while (cur > (next = F ? __ldca(p + cur) : cc_ld<H>(p + cur, pol))) {
       cc_st<H>(p + prev, next, pol);
       prev = cur;
       cur = next;
@@ -452,9 +455,9 @@ __device__ __forceinline__ uint32_t cc_find(uint32_t *p, uint32_t x, uint64_t po
   return cur;
 }
 
-template <bool H>
+template <bool H, bool F = false>
 __device__ __forceinline__ void cc_hook(uint32_t *p, uint32_t u, uint32_t v, uint64_t pol) {
-  uint32_t ru = cc_find<H>(p, u, pol), rv = cc_find<H>(p, v, pol);
+  uint32_t ru = cc_find<H, F>(p, u, pol), rv = cc_find<H, F>(p, v, pol);
   bool repeat;
   do {
     repeat = false;
@@ -511,7 +514,7 @@ __global__ void __launch_bounds__(TA) k_cc_sample(const uint64_t *__restrict__ k
 // Sample round over the rows (guard-indexed stores): each owned row hooks its first NS live
 // edges, found from row_offset (R8) -- slot row_offset[u] + 1 follows guard u-1 -- instead
 // of sweeping every slot; the scan skips a leaf's empty tail and stops at guard u.
-template <bool H, int NS>
+template <bool H, int NS, bool F = false>
 __global__ void __launch_bounds__(TA) k_cc_sample_rows(const uint64_t *__restrict__ key,
                                                        const uint32_t *__restrict__ tmask,
                                                        const uint64_t *__restrict__ row_offset, uint32_t L,
@@ -531,7 +534,7 @@ __global__ void __launch_bounds__(TA) k_cc_sample_rows(const uint64_t *__restric
       if ((__ldg(tmask + leaf_div(sl, L)) >> leaf_mod(sl, L)) & 1u) continue;   // tombstone
       const uint32_t v = (uint32_t)k;
       ++found;
-      if (u != v && cc_ld<H>(p + u, pol) != cc_ld<H>(p + v, pol)) cc_hook<H>(p, u, v, pol);
+      if (u != v && cc_ld<H>(p + u, pol) != cc_ld<H>(p + v, pol)) cc_hook<H, F>(p, u, v, pol);
     }
   }
 }
@@ -611,6 +614,12 @@ __global__ void __launch_bounds__(TA) k_cc_hook(const uint64_t *__restrict__ key
   }
 }
 
+// find() chain steps through L1 in the sampled round (GPMA_CC_L1, read per call)
+static bool cc_l1() {
+  const char *e = getenv("GPMA_CC_L1");
+  return !e || atoi(e) != 0;
+}
+
 static int cc_hint() {
   static const int v = [] { const char *e = getenv("GPMA_CC_HINT"); return e ? atoi(e) : 1; }();
   return v;
@@ -629,6 +638,8 @@ static cudaError_t cc_sample(gpma *g, uint32_t *p, cudaStream_t s) {
   if (g->rows_indexed && m > 0) {
     if (m == 1) GP_LAUNCH(g, (k_cc_sample_rows<true, 1>), grid_for(g->nr, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->row_offset, g->L,
                           g->nr, g->rb, p);
+    else if (cc_l1()) GP_LAUNCH(g, (k_cc_sample_rows<true, 2, true>), grid_for(g->nr, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask,
+                                g->row_offset, g->L, g->nr, g->rb, p);
     else GP_LAUNCH(g, (k_cc_sample_rows<true, 2>), grid_for(g->nr, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->row_offset, g->L,
                    g->nr, g->rb, p);
   } else if (cc_hint()) {
