@@ -579,7 +579,7 @@ __device__ __forceinline__ void cc_roots(uint32_t *p, uint32_t *out, uint32_t V)
 
 __global__ void k_cc_compress(uint32_t *p, uint32_t V) { cc_roots(p, p, V); }
 
-template <bool H>
+template <bool H, bool F = false>
 __device__ __forceinline__ void cc_group(const Slot4 &sl, uint32_t *p, uint64_t pol) {
   uint32_t pu[4], pv[4];
 #pragma unroll
@@ -594,11 +594,11 @@ __device__ __forceinline__ void cc_group(const Slot4 &sl, uint32_t *p, uint64_t 
   for (int j = 0; j < 4; ++j) {
     if (!edge4(sl, j) || pu[j] == pv[j]) continue;   // same tree already (fast path)
     uint32_t u = (uint32_t)(sl.k[j] >> 32), v = (uint32_t)sl.k[j];
-    if (u != v) cc_hook<H>(p, u, v, pol);
+    if (u != v) cc_hook<H, F>(p, u, v, pol);
   }
 }
 
-template <bool H>
+template <bool H, bool F = false>
 __global__ void __launch_bounds__(TA) k_cc_hook(const uint64_t *__restrict__ key,
                                                 const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
                                                 uint32_t *p) {
@@ -609,16 +609,18 @@ __global__ void __launch_bounds__(TA) k_cc_hook(const uint64_t *__restrict__ key
     const bool hb = t + stride < n4;
     load4(key, tmask, L, t * 4, a);
     if (hb) load4(key, tmask, L, (t + stride) * 4, b);
-    cc_group<H>(a, p, pol);
-    if (hb) cc_group<H>(b, p, pol);
+    cc_group<H, F>(a, p, pol);
+    if (hb) cc_group<H, F>(b, p, pol);
   }
 }
 
-// find() chain steps through L1 in the sampled round (GPMA_CC_L1, read per call)
-static bool cc_l1() {
+// find() chain steps through L1 (GPMA_CC_L1, read per call): 0 never, 1 sampled round,
+// 2 (default) sampled round and full pass
+static int cc_l1_mode() {
   const char *e = getenv("GPMA_CC_L1");
-  return !e || atoi(e) != 0;
+  return e ? atoi(e) : 2;
 }
+static bool cc_l1() { return cc_l1_mode() != 0; }
 
 static int cc_hint() {
   static const int v = [] { const char *e = getenv("GPMA_CC_HINT"); return e ? atoi(e) : 1; }();
@@ -675,7 +677,8 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
   GP_CHECK(g, cudaMemcpyAsync(prev, labels, V * 4, cudaMemcpyDeviceToDevice, s));
   GP_CHECK(g, cc_sample(g, labels, s));
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
-  if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
+  if (cc_l1_mode() >= 2) GP_LAUNCH(g, (k_cc_hook<true, true>), grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
+  else if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
   else GP_LAUNCH(g, k_cc_hook<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, labels);
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
   GP_CHECK(g, fill_zero(g, &X.ctrl_d->sum, 8, s));
@@ -696,7 +699,8 @@ gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s) {
   GP_LAUNCH(g, k_cc_init, grid_for(g->V), TA, 0, s, p, g->V);
   GP_CHECK(g, cc_sample(g, p, s));
   GP_LAUNCH(g, k_cc_compress, grid_for(g->V), TA, 0, s, p, g->V);
-  if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
+  if (cc_l1_mode() >= 2) GP_LAUNCH(g, (k_cc_hook<true, true>), grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
+  else if (cc_hint()) GP_LAUNCH(g, k_cc_hook<true>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
   else GP_LAUNCH(g, k_cc_hook<false>, grid_for(g->cap / 4, TA, SWEEP_BLOCKS), TA, 0, s, g->key, tmask, g->L, g->cap, p);
   GP_LAUNCH(g, k_cc_final, grid_for(g->V), TA, 0, s, p, labels, g->V);
   GP_CHECK(g, cudaGetLastError());

@@ -74,6 +74,7 @@ def test_cc_every_sample_strategy(scale):
     want = o.cc()
     from tests.gpu_helpers import gpu_cc
     for mode in ("0", "1", "2"):
-        with env(GPMA_CC_SAMPLE=mode):
-            got = gpu_cc(g)
-        assert np.array_equal(got, want), f"sample mode {mode}"
+        for l1 in ("0", "1", "2"):                      # find() chains through L1: never / sample / all
+            with env(GPMA_CC_SAMPLE=mode, GPMA_CC_L1=l1):
+                got = gpu_cc(g)
+            assert np.array_equal(got, want), f"sample mode {mode} L1 mode {l1}"
