@@ -120,8 +120,10 @@ class SlidingWindowPipeline:
                 torch.mul(self.x, 1.0, out=dx)
                 return it
 
-            def copies_now(st):
+            def copies_now(st, overlap=None):
                 self.ev_long.record(st)
+                if overlap is not None:    # enqueue the next (sync-free) kernels first: the copy
+                    overlap(st)            # issuing below then runs on the host while they do
                 self.xs.wait_event(self.ev_long)
                 self._flush_out(other)
                 self._flush_in(other)
@@ -134,8 +136,7 @@ class SlidingWindowPipeline:
                 it, n = r[0], r[3]
             else:
                 g.gpma_bfs(root, lv, stream=s)
-                copies_now(s)
-                g.gpma_cc(lab, stream=s)
+                copies_now(s, overlap=lambda st: g.gpma_cc(lab, stream=st))
                 it = pr(s)
                 n = g.gpma_export_csr(rp, col, cv, stream=s)
             self.pr_iters.append(it)
