@@ -817,7 +817,9 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
                                                     const uint32_t *__restrict__ tmask,
                                                     const uint64_t *__restrict__ head, uint32_t L, uint64_t cap,
                                                     const A *__restrict__ contrib, A *y, uint32_t rb,
-                                                    uint32_t nr, uint32_t dlo, uint32_t dhi, int hint) {
+                                                    uint32_t nr, uint32_t dlo, uint32_t dhi, int hint,
+                                                    const uint32_t *__restrict__ done) {
+  if (done && *done) return;                             // converged on the device (pagerank_t)
   const int lane = threadIdx.x & 31;
   uint64_t pol = 0;
   if (hint == 1) asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
@@ -878,7 +880,9 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
 template <typename T>
 __global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ y,
                           const uint32_t *__restrict__ deg, typename PrAcc<T>::A *__restrict__ contrib,
-                          uint32_t V, T d, const double *__restrict__ dsum_in, double *dsum_out, double *err) {
+                          uint32_t V, T d, const double *__restrict__ dsum_in, double *dsum_out, double *err,
+                          const uint32_t *__restrict__ done) {
+  if (*done) return;
   __shared__ double red[32];
   const T base = (T(1) - d) / T(V) + d * T(*dsum_in / (double)V);
   double e = 0, dl = 0;
@@ -917,6 +921,24 @@ __global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ 
   }
 }
 
+// Iteration bookkeeping on the device: zero the next error / dangling accumulators (first
+// kernel of an iteration), then, after the step, count the iteration and raise `done` once
+// the L1 change drops below tol (R20).  Every kernel of a later iteration returns
+// at once after `done`, so the host can queue iterations ahead and read back once per batch.
+struct PrLoop {
+  uint32_t done, iters;
+};
+__global__ void k_pr_iter_begin(double *acc, int nxt, const PrLoop *lp) {
+  if (lp->done || threadIdx.x) return;
+  acc[2] = 0.0;
+  acc[nxt] = 0.0;
+}
+__global__ void k_pr_iter_end(const double *acc, double tol, PrLoop *lp) {
+  if (lp->done || threadIdx.x) return;
+  lp->iters += 1;
+  if (acc[2] < tol) lp->done = 1;
+}
+
 // Destination passes of the push (GPMA_PR_PASSES, default 1).  Random REDs run ~3x faster
 // while their target fits in L2 (tools/micro/red_bench.cu), but each pass re-sweeps the keys;
 // at V = 2^24 one pass measured fastest.
@@ -943,33 +965,42 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   const uint64_t V = g->V;
   GP_CHECK(g, ensure(X.b[1], (V + 1) * sizeof(A), s));
   GP_CHECK(g, ensure(X.b[2], (V + 1) * sizeof(A), s));
-  GP_CHECK(g, ensure(X.b[3], 4 * sizeof(double), s));
+  GP_CHECK(g, ensure(X.b[3], 4 * sizeof(double) + sizeof(PrLoop), s));
   const uint32_t *deg = g->deg;
   A *contrib = (A *)X.b[1].p, *y = (A *)X.b[2].p;
-  double *acc = (double *)X.b[3].p;   // [0],[1] dangling ping-pong, [2] error
+  double *acc = (double *)X.b[3].p;   // [0],[1] dangling ping-pong, [2] error, then the loop state
+  PrLoop *lp = (PrLoop *)(acc + 4);
   const uint32_t passes = pr_passes(V * sizeof(A));
-  GP_CHECK(g, fill_zero(g, acc, 4 * sizeof(double), s));
+  GP_CHECK(g, fill_zero(g, acc, 4 * sizeof(double) + sizeof(PrLoop), s));
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
-  int it = 0, cur = 0;
-  while (it < max_iter) {
-    // destination passes: random REDs run ~3x faster while their target fits in L2
-    for (uint32_t q = 0; q < passes; ++q)
-      GP_LAUNCH(g, (k_pr_push_win<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
-                g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes),
-                pr_hint());
-    GP_CHECK(g, fill_zero(g, acc + 2, sizeof(double), s));
-    GP_CHECK(g, fill_zero(g, acc + (cur ^ 1), sizeof(double), s));
-    GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
-              acc + (cur ^ 1), acc + 2);
-    cur ^= 1;
-    ++it;
-    GP_CHECK(g, readback(g, &X.ctrl_h->sum2, acc + 2, 8, s));
+  // Iterations are queued in batches (2 first: a warm start rarely stops after one, then 1
+  // at a time) and gated on the device, so the common 2-3 iteration call reads back once or
+  // twice instead of once per iteration; the iterations that run are exactly those of the
+  // per-iteration host loop.
+  int queued = 0, cur = 0;
+  uint32_t it = 0;
+  while (queued < max_iter) {
+    const int batch = std::min(queued == 0 ? 2 : 1, max_iter - queued);
+    for (int b = 0; b < batch; ++b, ++queued) {
+      GP_LAUNCH(g, k_pr_iter_begin, 1, 32, 0, s, acc, cur ^ 1, lp);
+      // destination passes: random REDs run ~3x faster while their target fits in L2
+      for (uint32_t q = 0; q < passes; ++q)
+        GP_LAUNCH(g, (k_pr_push_win<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
+                  g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes),
+                  pr_hint(), &lp->done);
+      GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
+                acc + (cur ^ 1), acc + 2, &lp->done);
+      GP_LAUNCH(g, k_pr_iter_end, 1, 32, 0, s, acc, tol, lp);
+      cur ^= 1;
+    }
+    GP_CHECK(g, readback(g, &X.ctrl_h->sum2, lp, sizeof(PrLoop), s));
     GP_CHECK(g, cudaStreamSynchronize(s));
-    double e;
-    memcpy(&e, &X.ctrl_h->sum2, 8);
-    if (e < tol) break;
+    PrLoop h;
+    memcpy(&h, &X.ctrl_h->sum2, sizeof h);
+    it = h.iters;
+    if (h.done) break;
   }
-  if (iters) *iters = it;
+  if (iters) *iters = (int)it;
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
@@ -1026,7 +1057,7 @@ gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
   for (uint32_t q = 0; q < passes; ++q)
     GP_LAUNCH(g, (k_pr_push_win<unsigned long long, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g),
               g->head, g->L, g->cap, contrib, yy, g->rb, g->nr, (uint32_t)((uint64_t)g->V * q / passes),
-              (uint32_t)((uint64_t)g->V * (q + 1) / passes), pr_hint());
+              (uint32_t)((uint64_t)g->V * (q + 1) / passes), pr_hint(), nullptr);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
