@@ -142,6 +142,10 @@ def run_gpma(args, rank, world, lrank):
     need = args.warmup + 1 + args.steps + (0 if args.no_e2e else 2 * (1 + args.e2e_steps))
     assert need <= sw.n_slides, f"stream has {sw.n_slides} slides, need {need}"
     gen_s = time.time() - t0
+    torch.cuda.empty_cache()     # generator temporaries back to the device before the store allocates
+    # the generator's sort temporaries (tens of GB at P = 8) go back to the device before the
+    # store allocates (it does not draw from torch's cache)
+    torch.cuda.empty_cache()
     s = torch.cuda.Stream(dev)
     with torch.cuda.stream(s):
         k0, v0 = sw.initial()
@@ -427,6 +431,9 @@ def run_gpma_dist(args, rank, world, lrank):
     need = args.warmup + args.steps + (0 if args.no_e2e else 1 + args.e2e_steps)
     assert need <= sw.n_slides, f"stream has {sw.n_slides} slides, need {need}"
     gen_s = time.time() - t0
+    # the generator's sort temporaries (tens of GB at P = 8) go back to the device before the
+    # store allocates (it does not draw from torch's cache)
+    torch.cuda.empty_cache()
     s = torch.cuda.Stream(dev)
     rows = row_range(V, world, rank)
     bl, bh = batch_slice(B, world, rank)
@@ -639,8 +646,13 @@ def main():
     rank = int(os.environ.get("RANK", "0"))
     world = int(os.environ.get("WORLD_SIZE", "1"))
     lrank = int(os.environ.get("LOCAL_RANK", "0"))
+    # GPMA_BENCH_SHARE_GPU=1 (testing only): every rank on cuda:0 over gloo, to run the N > 1
+    # path on a one-GPU box (NCCL refuses two ranks per device)
+    share = os.environ.get("GPMA_BENCH_SHARE_GPU") == "1"
+    if share:
+        lrank = 0
     if world > 1 or args.force_dist:
-        backend = "nccl" if torch.cuda.is_available() else "gloo"
+        backend = "nccl" if torch.cuda.is_available() and not share else "gloo"
         if torch.cuda.is_available():
             torch.cuda.set_device(lrank)
         torch.distributed.init_process_group(backend)
