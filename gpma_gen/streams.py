@@ -114,6 +114,9 @@ def edge_values(keys: torch.Tensor, seed: int) -> torch.Tensor:
     return (_srl(draw(_tag(seed, 0x56414C), keys), 33) & 0x7FFFFFFF).to(torch.int32)
 
 
+_CUB_MAX = 1 << 30            # elements per sort/unique call (CUB takes < 2^31 items)
+
+
 def make_stream(kind: str, V: int, E: int, seed: int, scale: int | None = None,
                 device="cpu", sub_chunk: int = 1 << 27) -> torch.Tensor:
     """E unique edge keys (int64) in random-timestamp order.
@@ -121,14 +124,19 @@ def make_stream(kind: str, V: int, E: int, seed: int, scale: int | None = None,
     Draws candidates in rounds of max(E, 4096) until the set of unique, loop-free, in-range
     edges holds at least E keys; then orders that set by ts = draw(seed_ts, key) (signed
     int64 order, ties by key) and keeps the first E.  A round is generated in sub-chunks of
-    `sub_chunk` candidates to bound memory (this does not change the stream).
+    `sub_chunk` candidates to bound memory, and the set is kept in source-range buckets of
+    < 2^30 keys (sort limits at configs[4] scale, 2^31 edges); neither changes the stream.
     """
     new_id = _scramble(V, seed, device)
     chunk = max(E, 4096)
-    keys = torch.empty(0, dtype=torch.int64, device=device)
+    nbk = 1
+    while chunk * 2 // nbk > _CUB_MAX:                     # candidates per bucket per round
+        nbk *= 2
+    bnd = torch.tensor([((b * V) // nbk) << 32 for b in range(1, nbk)], dtype=torch.int64, device=device)
+    buckets = [torch.empty(0, dtype=torch.int64, device=device) for _ in range(nbk)]
     ctr = 0
-    while keys.numel() < E:
-        parts = [keys]
+    while sum(b.numel() for b in buckets) < E:
+        parts = [[b] for b in buckets]
         for c0 in range(ctr, ctr + chunk, sub_chunk):
             cn = min(sub_chunk, ctr + chunk - c0)
             if kind == "rmat":
@@ -139,16 +147,49 @@ def make_stream(kind: str, V: int, E: int, seed: int, scale: int | None = None,
                 raise ValueError(kind)
             ok = (s != d) & (s < V) & (d < V)
             s, d = new_id[s[ok]], new_id[d[ok]]
-            parts.append(torch.unique((s << 32) | d))
+            u = torch.unique((s << 32) | d)                  # sorted
             del s, d, ok
+            cut = [0] + torch.searchsorted(u, bnd).tolist() + [u.numel()]
+            for b in range(nbk):
+                parts[b].append(u[cut[b]:cut[b + 1]])
+            del u
         ctr += chunk
-        keys = torch.unique(torch.cat(parts))
+        for b in range(nbk):                                 # one bucket's temporaries at a time
+            buckets[b] = torch.unique(torch.cat(parts[b]))
+            parts[b] = None
         del parts
         if ctr > 64 * chunk:
             raise RuntimeError("stream generator: too few unique edges")
-    ts = draw(_tag(seed, 0x5453), keys)
-    order = torch.argsort(ts, stable=True)       # keys are sorted -> ties broken by key
-    return keys[order[:E]].contiguous()
+    keys = buckets[0] if nbk == 1 else torch.cat(buckets)    # sorted: buckets are key ranges
+    del buckets
+    tseed = _tag(seed, 0x5453)
+    if keys.numel() <= _CUB_MAX:
+        ts = draw(tseed, keys)
+        order = torch.argsort(ts, stable=True)               # keys are sorted -> ties broken by key
+        return keys[order[:E]].contiguous()
+    # above the sort limit: the 16 signed ranges of the top 4 bits of ts, in order, each sorted
+    # stably on its own (its keys stay in key order, so ties still break by key); ts is drawn
+    # in chunks and again per range, never held whole (its temporaries are 8 B per key each)
+    top = torch.empty(keys.numel(), dtype=torch.int8, device=keys.device)
+    for c0 in range(0, keys.numel(), _CUB_MAX // 4):
+        top[c0:c0 + _CUB_MAX // 4] = ((draw(tseed, keys[c0:c0 + _CUB_MAX // 4]) >> 60) + 8).to(torch.int8)
+    out = torch.empty(E, dtype=torch.int64, device=keys.device)
+    pos = 0
+    for b in range(16):
+        idx = torch.nonzero(top == b).squeeze(1)
+        if idx.numel() == 0:
+            continue
+        kr = keys[idx]
+        del idx
+        kb = kr[torch.argsort(draw(tseed, kr), stable=True)]
+        del kr
+        take = min(kb.numel(), E - pos)
+        out[pos:pos + take] = kb[:take]
+        pos += take
+        del kb
+        if pos == E:
+            break
+    return out
 
 
 def weak_scaled(cfg_index: int, P: int) -> "StreamConfig":

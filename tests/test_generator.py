@@ -28,3 +28,16 @@ def test_stream_config0_shape():
     assert torch.equal(config_stream(0).keys, k)
     d = draw(1, torch.arange(4))
     assert torch.equal(d, draw(1, torch.arange(4)))
+
+
+def test_bucketed_generation_is_the_same_stream(monkeypatch):
+    """Above the sort limit (configs[4]: 2^31 edges) the generator keeps the edge set in
+    source-range buckets and sorts timestamps by ranges; forced here at small sizes, the stream
+    must be identical to the single-sort one."""
+    import gpma_gen.streams as S
+    ref = S.make_stream("rmat", 1 << 12, 40000, 7, scale=12)
+    ref_u = S.make_stream("uniform", 5000, 30000, 3)
+    # (a range of the split timestamp sort must itself fit: 40000 keys / 16 ranges < 2^12)
+    monkeypatch.setattr(S, "_CUB_MAX", 1 << 12)
+    assert torch.equal(S.make_stream("rmat", 1 << 12, 40000, 7, scale=12, sub_chunk=1 << 11), ref)
+    assert torch.equal(S.make_stream("uniform", 5000, 30000, 3, sub_chunk=1 << 12), ref_u)
