@@ -586,8 +586,14 @@ __device__ __forceinline__ void cc_group(const Slot4 &sl, uint32_t *p, uint64_t 
   for (int j = 0; j < 4; ++j) {             // independent parent loads first
     pu[j] = pv[j] = 0;
     if (edge4(sl, j)) {
-      pu[j] = cc_ld<H>(p + (uint32_t)(sl.k[j] >> 32), pol);
-      pv[j] = cc_ld<H>(p + (uint32_t)sl.k[j], pol);
+      if (F) {            // same-tree filter through L1: a stale parent is an ancestor, so equal
+                          // parents still prove one tree; a miss costs the exact find + CAS
+        pu[j] = __ldca(p + (uint32_t)(sl.k[j] >> 32));
+        pv[j] = __ldca(p + (uint32_t)sl.k[j]);
+      } else {
+        pu[j] = cc_ld<H>(p + (uint32_t)(sl.k[j] >> 32), pol);
+        pv[j] = cc_ld<H>(p + (uint32_t)sl.k[j], pol);
+      }
     }
   }
 #pragma unroll
