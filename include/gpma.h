@@ -223,6 +223,23 @@ gpma_status gpma_pr_push(gpma_t *g, double *x, int init, uint64_t *y, gpma_strea
 /* x'[v] = (1-d)/V + d*(y[v] + y[V]/V) for every v; *err (HOST) = ||x'-x||_1; y := 0. */
 gpma_status gpma_pr_update(gpma_t *g, double *x, uint64_t *y, double damping, double *err,
                            gpma_stream_t stream);
+/* The same update for the OWNED rows only, after a reduce-scatter of the pushes (SURVEY
+ * §8(e)): y_rows[0..nr) (device) = the summed y of rows [row_begin, row_end), y_rows[nr] = the
+ * total dangling mass (2^-62 units); x[row_begin + i] := (1-d)/V + d*(y_rows[i] + y_rows[nr]/V);
+ * *err (HOST) = the owned rows' part of ||x'-x||_1 (sum it over the ranks).  y_rows is not
+ * modified; x outside the owned rows is not touched (all-gather the owned slices for the full
+ * vector).  P:1215-1227. */
+gpma_status gpma_pr_update_rows(gpma_t *g, double *x, const uint64_t *y_rows, double damping, double *err,
+                                gpma_stream_t stream);
+/* Multi-GPU BFS exchange ("synchronize all devices after each
+ * iteration"): bitmap[ceil(V/32)] (device) := bit v set iff levels[v] == depth, i.e. this
+ * rank's discoveries of the level just expanded.  Ranks all-gather their bitmaps (V/8 bytes
+ * each instead of an all-reduce of 4V-byte levels). */
+gpma_status gpma_bfs_bits(gpma_t *g, const int32_t *levels, int32_t depth, uint32_t *bitmap, gpma_stream_t stream);
+/* levels[v] := depth where levels[v] == -1 and bit v is set in any of the nbitmaps bitmaps
+ * laid out back to back (ceil(V/32) words each, device).  After it, levels are replicated. */
+gpma_status gpma_bfs_merge(gpma_t *g, int32_t *levels, const uint32_t *bitmaps, uint32_t nbitmaps, int32_t depth,
+                           gpma_stream_t stream);
 
 /* Kernel profiler (bench evidence, CUDA events on the call's stream around each launch):
  * filter NULL/"" = off, "*" = every kernel, else one kernel name (e.g. "k_pr_push").

@@ -367,6 +367,38 @@ static gpma_status bfs_expand_level(gpma *g, Scratch &X, int32_t *levels, int32_
   return GPMA_OK;
 }
 
+// Multi-GPU BFS exchange: a rank's discoveries of one level as a bitmap
+// (bit v = levels[v] == depth), and the merge of every rank's bitmap into levels.
+__global__ void k_bfs_bits(const int32_t *__restrict__ levels, uint32_t V, int32_t d, uint32_t *__restrict__ bm) {
+  const uint64_t Vr = ((uint64_t)V + 31) & ~31ull;
+  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < Vr; v += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t b = __ballot_sync(0xffffffffu, v < V && levels[v] == d);
+    if ((threadIdx.x & 31) == 0) bm[v >> 5] = b;
+  }
+}
+
+__global__ void k_bfs_merge(int32_t *__restrict__ levels, uint32_t V, const uint32_t *__restrict__ bms,
+                            uint32_t nbm, uint64_t words, int32_t d) {
+  for (uint64_t v = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; v < V; v += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t any = 0;
+    for (uint32_t r = 0; r < nbm; ++r) any |= __ldg(bms + r * words + (v >> 5));
+    if (((any >> (v & 31)) & 1u) && levels[v] == -1) levels[v] = d;
+  }
+}
+
+gpma_status bfs_bits(gpma *g, const int32_t *levels, int32_t depth, uint32_t *bm, cudaStream_t s) {
+  GP_LAUNCH(g, k_bfs_bits, grid_for(((uint64_t)g->V + 31) & ~31ull), TA, 0, s, levels, g->V, depth, bm);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+gpma_status bfs_merge(gpma *g, int32_t *levels, const uint32_t *bms, uint32_t nbm, int32_t depth, cudaStream_t s) {
+  const uint64_t words = ((uint64_t)g->V + 31) / 32;
+  GP_LAUNCH(g, k_bfs_merge, grid_for(g->V), TA, 0, s, levels, g->V, bms, nbm, words, depth);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 // One BFS level of a (possibly sharded) store: the frontier is {v : levels[v] == depth-1}
 // (levels may be replicated across shards); the owned rows of the frontier are expanded and
 // newly reached vertices get `depth`.  *frontier = the frontier size (0: nothing expanded).
@@ -1075,6 +1107,37 @@ gpma_status pr_update(gpma *g, double *x, uint64_t *y, double d, double *err, cu
   GP_CHECK(g, fill_zero(g, e_d, 8, s));
   GP_LAUNCH(g, k_prd_update, grid_for(g->V), TA, 0, s, x, (unsigned long long *)y, g->V, d, e_d);
   GP_CHECK(g, fill_zero(g, y + g->V, 8, s));
+  GP_CHECK(g, readback(g, &X.ctrl_h->sum2, e_d, 8, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  memcpy(err, &X.ctrl_h->sum2, 8);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
+// Owned-rows update after a reduce-scatter of y (multi-GPU): y_rows[0..nr) =
+// the summed pushes into the owned vertices, y_rows[nr] = the total dangling mass.
+// x'[rb+i] = (1-d)/V + d (y_rows[i] + y_rows[nr]/V); err = sum |x'-x| over the owned rows.
+__global__ void k_prd_update_rows(double *__restrict__ x, const unsigned long long *__restrict__ yr, uint32_t rb,
+                                  uint32_t nr, uint32_t V, double d, double *err) {
+  __shared__ double red[32];
+  const double base = (1.0 - d) / (double)V + d * (PrAcc<double>::dec(yr[nr]) / (double)V);
+  double e = 0;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < nr; i += (uint64_t)gridDim.x * blockDim.x) {
+    const double nx = base + d * PrAcc<double>::dec(yr[i]);
+    e += fabs(nx - x[rb + i]);
+    x[rb + i] = nx;
+  }
+  double se = block_sum_d(e, red);
+  if (threadIdx.x == 0 && se != 0) atomicAdd(err, se);
+}
+
+gpma_status pr_update_rows(gpma *g, double *x, const uint64_t *y_rows, double d, double *err, cudaStream_t s) {
+  Scratch &X = g->an[AN_PR];
+  ScanScope scan_scope_(X.scan);
+  double *e_d = reinterpret_cast<double *>(&X.ctrl_d->sum2);
+  GP_CHECK(g, fill_zero(g, e_d, 8, s));
+  GP_LAUNCH(g, k_prd_update_rows, grid_for(g->nr), TA, 0, s, x, (const unsigned long long *)y_rows, g->rb, g->nr,
+            g->V, d, e_d);
   GP_CHECK(g, readback(g, &X.ctrl_h->sum2, e_d, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   memcpy(err, &X.ctrl_h->sum2, 8);

@@ -576,6 +576,29 @@ gpma_status gpma_pr_update(gpma_t *g, double *x, uint64_t *y, double damping, do
   return end(g, gp::pr_update(g, x, y, damping, err, (cudaStream_t)stream));
 }
 
+gpma_status gpma_pr_update_rows(gpma_t *g, double *x, const uint64_t *y_rows, double damping, double *err,
+                                gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!x || !y_rows || !err || !(damping >= 0.0 && damping <= 1.0)) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::pr_update_rows(g, x, y_rows, damping, err, (cudaStream_t)stream));
+}
+
+gpma_status gpma_bfs_bits(gpma_t *g, const int32_t *levels, int32_t depth, uint32_t *bitmap, gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!levels || !bitmap) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::bfs_bits(g, levels, depth, bitmap, (cudaStream_t)stream));
+}
+
+gpma_status gpma_bfs_merge(gpma_t *g, int32_t *levels, const uint32_t *bitmaps, uint32_t nbitmaps, int32_t depth,
+                           gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!levels || (nbitmaps && !bitmaps) || depth < 1) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::bfs_merge(g, levels, bitmaps, nbitmaps, depth, (cudaStream_t)stream));
+}
+
 uint64_t gpma_kernel_launches(const gpma_t *g) { return g ? g->launches.load() : 0; }
 
 const char *gpma_status_string(gpma_status s) {

@@ -12,12 +12,15 @@ caller's torch.distributed process group (NCCL over NVLink on B200; gloo in the 
 * update: each rank routes its contiguous slice of the global batch by owner (stable) and an
   all-to-all-v delivers the pieces; the rank-order concatenation keeps the global batch order,
   so "last occurrence wins" (R10) is preserved.
-* BFS: levels are replicated; each level expands the owned frontier rows, then MAX-all-reduce.
+* BFS: levels are replicated; each level expands the owned frontier rows, then the ranks
+  all-gather their discoveries as bitmaps (V/8 bytes each) and merge them into levels.
 * CC: labels are replicated; each round hooks the owned edges on top of them, then
   MIN-all-reduce; stop when no rank changed anything (fixpoint = min-id labels, R19).
-* PageRank: x is replicated; each iteration pushes the owned rows into an exact 64-bit
-  fixed-point y (plus the owned dangling mass), SUM-all-reduces it, and every rank applies the
-  same update -- so x stays bit-identical across ranks.
+* PageRank: each iteration pushes the owned rows into an exact 64-bit fixed-point y (plus the
+  owned dangling mass), REDUCE-SCATTERs y to the owners (half an all-reduce's traffic), and
+  each rank updates only its owned slice of x (the only one its next push reads); the error
+  and the dangling mass are two-word all-reduces; an all-gather of the owned slices returns the
+  full vector at the end.
 """
 from __future__ import annotations
 
@@ -88,6 +91,15 @@ class CudaShard:
     def pr_update(self, x, y, damping) -> float:
         return self.g.gpma_pr_update(x, y, damping, stream=self.stream)
 
+    def pr_update_rows(self, x, y_rows, damping) -> float:
+        return self.g.gpma_pr_update_rows(x, y_rows, damping, stream=self.stream)
+
+    def bfs_bits(self, levels, depth, bitmap):
+        self.g.gpma_bfs_bits(levels, depth, bitmap, stream=self.stream)
+
+    def bfs_merge(self, levels, bitmaps, n, depth):
+        self.g.gpma_bfs_merge(levels, bitmaps, n, depth, stream=self.stream)
+
     def sync(self):
         if self.device.type == "cuda":
             (self.stream or torch.cuda.current_stream(self.device)).synchronize()
@@ -124,6 +136,28 @@ class DistGpma:
         dist.all_reduce(h, op=op, group=self.group)
         return self._back(h, t)
 
+    def _all_gather(self, out, t):
+        """out (P * t.numel()) := the ranks' t, back to back."""
+        if self.P == 1:
+            out.copy_(t)
+            return out
+        if self._cpu_coll:                  # gloo: list all-gather of host copies
+            parts = [torch.empty_like(self._dev(t)) for _ in range(self.P)]
+            dist.all_gather(parts, self._dev(t).contiguous(), group=self.group)
+            return self._back(torch.cat(parts), out)
+        dist.all_gather_into_tensor(out, t.contiguous(), group=self.group)
+        return out
+
+    def _reduce_scatter(self, out, t):
+        """out (t.numel() / P) := this rank's slice of the element-wise SUM of the ranks' t."""
+        if self._cpu_coll:                  # gloo has no reduce-scatter: all-reduce, keep the slice
+            h = self._dev(t).clone()
+            dist.all_reduce(h, group=self.group)
+            n = out.numel()
+            return self._back(h[self.r * n:(self.r + 1) * n], out)
+        dist.reduce_scatter_tensor(out, t, group=self.group)
+        return out
+
     def _exchange(self, keys, vals):
         """Route this rank's slice by owner and all-to-all-v it: returns the owned batch."""
         if self.P == 1:
@@ -158,12 +192,18 @@ class DistGpma:
     def bfs(self, root: int, levels=None):
         levels = self.shard.vertex_array(self.V, torch.int32) if levels is None else levels
         self.shard.bfs_init(root, levels)
+        words = (self.V + 31) // 32
+        bm = self.shard.vertex_array(words, torch.int32)
+        bms = self.shard.vertex_array(self.P * words, torch.int32)
         depth = 1
         while True:
-            F = self.shard.bfs_level(levels, depth)
+            F = self.shard.bfs_level(levels, depth)      # |frontier| of the replicated levels
             if F == 0:
                 break
-            self._all_reduce(levels, dist.ReduceOp.MAX)
+            if self.P > 1:
+                self.shard.bfs_bits(levels, depth, bm)   # this rank's discoveries
+                self._all_gather(bms, bm)
+                self.shard.bfs_merge(levels, bms, self.P, depth)
             depth += 1
         return levels
 
@@ -187,14 +227,40 @@ class DistGpma:
     def pagerank(self, x=None, warm: bool = False, damping: float = 0.85, tol: float = 1e-3,
                  max_iter: int = 100):
         x = self.shard.vertex_array(self.V, torch.float64) if x is None else x
-        y = self.shard.vertex_array(self.V + 1, torch.int64)
-        y.zero_()
         it = 0
+        if self.P == 1:
+            y = self.shard.vertex_array(self.V + 1, torch.int64)
+            y.zero_()
+            while it < max_iter:
+                self.shard.pr_push(x, (not warm) and it == 0, y)
+                err = self.shard.pr_update(x, y, damping)
+                it += 1
+                if err < tol:
+                    break
+            return x, it
+        chunk = (self.V + self.P - 1) // self.P
+        lo, hi = self.rows
+        y = self.shard.vertex_array(chunk * self.P + 1, torch.int64)   # y[V] = dangling mass
+        yr = self.shard.vertex_array(chunk + 1, torch.int64)          # owned sums, then the dangling total
+        e = self.shard.vertex_array(1, torch.float64)
+        y.zero_()
         while it < max_iter:
             self.shard.pr_push(x, (not warm) and it == 0, y)
-            self._all_reduce(y, dist.ReduceOp.SUM)
-            err = self.shard.pr_update(x, y, damping)
+            self._reduce_scatter(yr[:chunk], y[:chunk * self.P])
+            dang = y[self.V:self.V + 1].clone()
+            self._all_reduce(dang, dist.ReduceOp.SUM)
+            yr[hi - lo:hi - lo + 1].copy_(dang)
+            e.fill_(self.shard.pr_update_rows(x, yr, damping))
+            self._all_reduce(e, dist.ReduceOp.SUM)
+            y.zero_()
             it += 1
-            if err < tol:
+            if float(e.item()) < tol:
                 break
+        # replicate x: the owned slices, back to back (the last one padded to chunk)
+        xs = self.shard.vertex_array(chunk * self.P, torch.float64)
+        mine = self.shard.vertex_array(chunk, torch.float64)
+        mine.zero_()
+        mine[:hi - lo].copy_(x[lo:hi])
+        self._all_gather(xs, mine)
+        x.copy_(xs[:self.V])
         return x, it

@@ -82,6 +82,9 @@ def lib() -> C.CDLL:
             "gpma_cc_round": (st, [P, P, i32, P, P]),
             "gpma_pr_push": (st, [P, P, i32, P, P]),
             "gpma_pr_update": (st, [P, P, P, C.c_double, P, P]),
+            "gpma_pr_update_rows": (st, [P, P, P, C.c_double, P, P]),
+            "gpma_bfs_bits": (st, [P, P, i32, P, P]),
+            "gpma_bfs_merge": (st, [P, P, P, u32, i32, P]),
             "gpma_debug_profile": (st, [P, C.c_char_p]),
             "gpma_debug_profile_read": (st, [P, C.c_char_p, C.c_size_t]),
             "gpma_status_string": (C.c_char_p, [st]),
@@ -98,7 +101,8 @@ EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destro
            "gpma_bfs", "gpma_cc", "gpma_pagerank", "gpma_pagerank_f32", "gpma_export_csr", "gpma_stats",
            "gpma_debug_dump", "gpma_debug_set_trace", "gpma_debug_trace", "gpma_kernel_launches",
            "gpma_debug_profile", "gpma_debug_profile_read", "gpma_route", "gpma_bfs_init", "gpma_bfs_level",
-           "gpma_cc_round", "gpma_pr_push", "gpma_pr_update", "gpma_query_edges", "gpma_query_neighbors",
+           "gpma_cc_round", "gpma_pr_push", "gpma_pr_update", "gpma_pr_update_rows", "gpma_bfs_bits",
+           "gpma_bfs_merge", "gpma_query_edges", "gpma_query_neighbors",
            "gpma_query_reachable",
            "gpma_status_string", "gpma_last_error"]
 
@@ -315,6 +319,20 @@ class Gpma:
         self._check(lib().gpma_pr_update(self._h, _ptr(x), _ptr(y), damping, C.byref(e), _stream(stream)),
                     "gpma_pr_update")
         return e.value
+
+    def gpma_pr_update_rows(self, x, y_rows, damping: float = 0.85, stream=None) -> float:
+        e = C.c_double(0.0)
+        self._check(lib().gpma_pr_update_rows(self._h, _ptr(x), _ptr(y_rows), damping, C.byref(e),
+                                              _stream(stream)), "gpma_pr_update_rows")
+        return e.value
+
+    def gpma_bfs_bits(self, levels, depth: int, bitmap, stream=None):
+        self._check(lib().gpma_bfs_bits(self._h, _ptr(levels), depth, _ptr(bitmap), _stream(stream)),
+                    "gpma_bfs_bits")
+
+    def gpma_bfs_merge(self, levels, bitmaps, nbitmaps: int, depth: int, stream=None):
+        self._check(lib().gpma_bfs_merge(self._h, _ptr(levels), _ptr(bitmaps), nbitmaps, depth, _stream(stream)),
+                    "gpma_bfs_merge")
 
     def gpma_kernel_launches(self) -> int:
         return int(lib().gpma_kernel_launches(self._h))

@@ -114,3 +114,31 @@ class OracleShard:
         xv[:] = nx
         yy[:] = 0
         return err
+
+    def pr_update_rows(self, x, y_rows, damping):
+        """gpma_pr_update_rows: the owned rows from their reduced sums (+ y_rows[nr] = dangling)."""
+        xv = x.numpy()
+        yr = y_rows.numpy().view(np.uint64)
+        lo, hi = self.rows
+        nr = hi - lo
+        D = float(yr[nr]) / SCALE
+        nx = (1 - damping) / self.V + damping * (yr[:nr].astype(np.float64) / SCALE + D / self.V)
+        err = float(np.abs(nx - xv[lo:hi]).sum())
+        xv[lo:hi] = nx
+        return err
+
+    def bfs_bits(self, levels, depth, bitmap):
+        """gpma_bfs_bits: bit v of bitmap = (levels[v] == depth)."""
+        lv = levels.numpy()
+        bits = np.zeros(bitmap.numel() * 32, dtype=np.uint8)
+        bits[: self.V] = lv == depth
+        bitmap.numpy().view(np.uint32)[:] = np.packbits(bits, bitorder="little").view(np.uint32)
+
+    def bfs_merge(self, levels, bitmaps, n, depth):
+        """gpma_bfs_merge: levels[v] := depth where unreached and set in any bitmap."""
+        lv = levels.numpy()
+        words = (self.V + 31) // 32
+        b = bitmaps.numpy().view(np.uint32).reshape(n, words)
+        anyb = np.bitwise_or.reduce(b, axis=0)
+        bits = np.unpackbits(anyb.view(np.uint8), bitorder="little")[: self.V].astype(bool)
+        lv[bits & (lv == -1)] = depth
