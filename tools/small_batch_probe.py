@@ -16,16 +16,16 @@ sw = config_stream(1, device=dev)
 k0, v0 = sw.initial()
 s = torch.cuda.Stream(dev)
 with torch.cuda.stream(s):
-    for B in (100, 1000, 10000):
+    for B in [int(b) for b in (sys.argv[1:] or ["100", "1000", "10000"])]:
         g = Gpma.gpma_create(1_600_000, k0.contiguous(), v0.contiguous(), stream=s)
         pos = 0
         ev, hd, hi = [], [], []
-        for it in range(60):
+        for it in range(min(60, (sw.keys.numel() - sw.window) // B - 1)):
             dk = sw.keys[pos:pos + B]
             ik = sw.keys[sw.window + pos: sw.window + pos + B]
             iv = sw.vals[sw.window + pos: sw.window + pos + B]
             pos += B
-            if it == 50:
+            if it == min(50, (sw.keys.numel() - sw.window) // B - 3):
                 g.gpma_debug_profile("*")
             e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
             e0.record(s)
@@ -36,14 +36,14 @@ with torch.cuda.stream(s):
             t2 = time.perf_counter()
             e1.record(s)
             e1.synchronize()
-            if it == 50:
+            if it == min(50, (sw.keys.numel() - sw.window) // B - 3):
                 prof = g.gpma_debug_profile_read()
                 g.gpma_debug_profile(None)
-            elif it >= 10:
+            elif it >= 3:
                 ev.append(e0.elapsed_time(e1))
                 hd.append((t1 - t0) * 1e3)
                 hi.append((t2 - t1) * 1e3)
-        print(f"B={B}: slide {np.mean(ev):.4f} ms (events), host delete call {np.mean(hd):.4f} ms, "
+        print(f"B={B}: levels climbed by the last insert {g.gpma_stats()['last_top_level']}; slide {np.mean(ev):.4f} ms (events), host delete call {np.mean(hd):.4f} ms, "
               f"host insert call {np.mean(hi):.4f} ms")
         tot = sum(v[1] for v in prof.values())
         n = sum(v[0] for v in prof.values())
