@@ -118,11 +118,11 @@ def algo_bytes(kernel: str, cap: int, V: int, L: int, nnz: int, dtype_bytes: int
     """Algorithmic bytes of ONE launch, from SURVEY.md §8(d)'s per-unit figures (keys 8 B +
     values 4 B per slot): PR push 12·cap + 8·V + 8·E per iteration; CC hooking round
     12·cap + 8·E; export 12·cap + 8·(V+1) + 8·E.  E = live edges."""
-    if kernel in ("k_pr_push", "k_pr_push_win", "k_pr_push_tma"):    # slots, x/outdeg per row, scatter-add y[dst]
+    if kernel == "k_pr_push_win":       # slots, x/outdeg per row, scatter-add y[dst]
         return 12 * cap + 8 * V + 8 * nnz
     if kernel in ("k_cc_hook", "k_cc_sample"):     # one hooking sweep
         return 12 * cap + 8 * nnz
-    if kernel == "k_exp_write":
+    if kernel in ("k_exp_write", "k_exp_tma"):
         return 12 * cap + 8 * (V + 1) + 8 * nnz
     return None
 

@@ -794,47 +794,6 @@ __global__ void k_pr_prep(T *__restrict__ x, const uint32_t *__restrict__ deg,
   if (threadIdx.x == 0 && s != 0) atomicAdd(dsum, s);
 }
 
-// y[v] += contrib[u] over the live edges u -> v (push SpMV): two groups of 4 slots per
-// thread, all loads (keys, masks, contributions) issued before the fire-and-forget REDs.
-template <typename A>
-__device__ __forceinline__ void pr_contribs(const Slot4 &sl, const A *__restrict__ contrib, A cv[4], uint32_t rb) {
-  uint32_t cu = 0xFFFFFFFFu;
-  A c = 0;
-#pragma unroll
-  for (int j = 0; j < 4; ++j) {
-    cv[j] = 0;
-    if (!edge4(sl, j)) continue;
-    uint32_t u = (uint32_t)(sl.k[j] >> 32) - rb;     // contributions are per owned row
-    if (u != cu) { cu = u; c = __ldcs(contrib + u); }
-    cv[j] = c;
-  }
-}
-
-template <typename A>
-__device__ __forceinline__ void pr_scatter(const Slot4 &sl, const A cv[4], A *y) {
-#pragma unroll
-  for (int j = 0; j < 4; ++j)
-    if (edge4(sl, j)) atomicAdd(&y[(uint32_t)sl.k[j]], cv[j]);
-}
-
-template <typename A>
-__global__ void __launch_bounds__(TA) k_pr_push(const uint64_t *__restrict__ key,
-                                                const uint32_t *__restrict__ tmask, uint32_t L, uint64_t cap,
-                                                const A *__restrict__ contrib, A *y, uint32_t rb) {
-  const uint64_t n4 = cap / 4, stride = (uint64_t)gridDim.x * blockDim.x;
-  for (uint64_t t = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; t < n4; t += 2 * stride) {
-    Slot4 a, b;
-    const bool hb = t + stride < n4;
-    load4(key, tmask, L, t * 4, a);
-    if (hb) load4(key, tmask, L, (t + stride) * 4, b);
-    A ca[4], cb[4];
-    pr_contribs(a, contrib, ca, rb);
-    if (hb) pr_contribs(b, contrib, cb, rb);
-    pr_scatter(a, ca, y);
-    if (hb) pr_scatter(b, cb, y);
-  }
-}
-
 // RED with an L2 eviction-priority hint (evict_last keeps the scattered y lines resident
 // while the key stream, loaded evict-first, passes through L2).
 __device__ __forceinline__ void red_add_hint(unsigned long long *p, unsigned long long v, uint64_t pol) {
