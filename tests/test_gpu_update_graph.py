@@ -94,3 +94,40 @@ def test_graph_replay_errors_and_launch_accounting():
         s.synchronize()
         o.insert(b + np.uint64(1), np.full(5, 7, dtype=np.uint32))
         assert_same_layout(g, o, what="plain launches")
+
+
+@pytest.mark.parametrize("mode", [0, 1])
+@pytest.mark.parametrize("seed", range(6))
+def test_graph_replay_across_resizes(seed, mode):
+    """Fixed-size random insert / delete batches on a side stream (so the prefix graph is
+    captured and replayed) on tiny graphs whose capacity doubles and halves: a resize changes
+    the signature (store pointers, geometry), the graph is dropped and re-captured; layouts
+    must equal the oracle after every batch."""
+    rng = np.random.default_rng(100 + seed)
+    V = int(rng.integers(16, 48))
+    n0 = 4 * V
+    k0 = [(int(a) << 32) | int(b) for a, b in zip(rng.integers(0, V, n0), rng.integers(0, V, n0))]
+    v0 = rng.integers(0, 1 << 31, n0).tolist()
+    s = torch.cuda.Stream(DEV)
+    with torch.cuda.stream(s):
+        g = Gpma.gpma_create(V, keys_t(k0), vals_t(v0), delete_mode=mode, stream=s)
+    o = O.Oracle(V, k0, v0, delete_mode=mode)
+    live = set(k0)
+    B = 2 * V                                   # one batch size for every op: replayable
+    for step in range(40):
+        grow = (step // 10) % 2 == 0
+        if grow or not live:
+            ks = [(int(a) << 32) | int(b) for a, b in zip(rng.integers(0, V, B), rng.integers(0, V, B))]
+            vs = rng.integers(0, 1 << 31, B).tolist()
+            g.gpma_update_batch(keys_t(ks), vals_t(vs), 0, stream=s)
+            o.insert(ks, vs)
+            live.update(ks)
+        else:
+            pres = sorted(live)
+            ks = [pres[i] for i in rng.integers(0, len(pres), B)]
+            g.gpma_update_batch(keys_t(ks), None, 1, stream=s)
+            o.delete(ks)
+            live.difference_update(ks)
+        s.synchronize()
+        assert_same_layout(g, o, what=f"seed {seed} step {step}")
+    assert_same_csr(g, o)
