@@ -55,6 +55,7 @@ def parse():
     ap.add_argument("--profile-all", action="store_true", help="print the per-kernel time table")
     ap.add_argument("--force-dist", action="store_true", help="use the sharded path even at N=1 (testing)")
     ap.add_argument("--no-sweep", action="store_true", help="skip the configs[1] batch-size sweep")
+    ap.add_argument("--no-resize", action="store_true", help="skip the configs[3] grow/shrink resize stress")
     ap.add_argument("--concurrent-analytics", action="store_true",
                     help="run BFS/CC/PR/export side by side on 4 streams (fanout.py) instead of one "
                          "after another (the default: per-phase breakdown, uncontended roofline)")
@@ -362,9 +363,81 @@ def run_gpma(args, rank, world, lrank):
         del sw, g
         torch.cuda.empty_cache()
         out["batch_sweep"] = batch_sweep(dev)
+    if not args.no_resize:
+        torch.cuda.empty_cache()
+        out["resize_stress"] = resize_stress(dev)
+        torch.cuda.empty_cache()
     if world == 1 and not args.no_cpu_baseline:
         out["cpu_baseline"] = cpu_baseline(config_stream(args.config, device=dev), cfg, args, 0)
     print(json.dumps(out))
+
+
+def resize_stress(dev, grow_steps=242, shrink_steps=248):
+    """configs[3]: V = 2^24, a pool of 2^28 unique uniform edges, strict
+    (rebalancing) deletes.  Start with 2^23 live edges; grow with (INSERT 2^20 new, DELETE 2^18
+    oldest) x 242, then shrink with (INSERT 2^18, DELETE 2^20 oldest) x 248 -- the live set is a
+    FIFO over the pool, which is recycled from its start once used up (those keys were deleted
+    long before).  Capacity doubles on the way up and halves on the way down (Alg. 4 l.16-17,
+    R14).  CUDA events per step (insert + delete); steps that resized are reported apart."""
+    from paper_journals_pvldb_shalht17_b200 import Gpma
+    from gpma_gen.streams import edge_values, make_stream
+    cfg = CONFIGS[3]
+    V = cfg.V
+    t0 = time.time()
+    pool = make_stream("uniform", V, cfg.E, cfg.seed, device=dev)
+    vals = edge_values(pool, cfg.seed)
+    torch.cuda.synchronize()
+    gen_s = time.time() - t0
+    torch.cuda.empty_cache()
+    N = pool.numel()
+
+    def seq(a, b):                          # FIFO positions [a, b) -> pool keys (recycled)
+        idx = torch.arange(a, b, device=dev) % N
+        return pool[idx].contiguous(), vals[idx].contiguous()
+
+    s = torch.cuda.Stream(dev)
+    f, b = 0, 1 << 23
+    with torch.cuda.stream(s):
+        k0, v0 = seq(f, b)
+        g = Gpma.gpma_create(V, k0, v0, delete_mode=1, stream=s)
+        del k0, v0
+        st = g.gpma_stats()
+        cap0, res0 = st["capacity"], st["resizes"]
+        caps, times, resized = [cap0], [], []
+        upd = 0
+        for step in range(grow_steps + shrink_steps):
+            ni, nd = (1 << 20, 1 << 18) if step < grow_steps else (1 << 18, 1 << 20)
+            nd = min(nd, b + ni - f)
+            ik, iv = seq(b, b + ni)
+            dk, _ = seq(f, f + nd)
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record(s)
+            g.gpma_update_batch(ik, iv, 0, stream=s)
+            g.gpma_update_batch(dk, None, 1, stream=s)
+            e1.record(s)
+            e1.synchronize()
+            b += ni
+            f += nd
+            upd += ni + nd
+            st = g.gpma_stats()
+            times.append(e0.elapsed_time(e1))
+            resized.append(st["resizes"] != res0)
+            res0 = st["resizes"]
+            caps.append(st["capacity"])
+        live = g.gpma_stats()["live_edges"]
+        del g
+    t = np.array(times)
+    rz = np.array(resized)
+    dbl = sum(1 for a, c in zip(caps, caps[1:]) if c > a)
+    hlv = sum(1 for a, c in zip(caps, caps[1:]) if c < a)
+    return {"workload": "configs[3] uniform V=2^24, 2^28-edge pool, strict deletes: 242 grow + 248 shrink steps",
+            "updates_per_s": upd / (t.sum() / 1e3), "ms_per_step_mean": float(t.mean()),
+            "steps": int(t.size), "resize_steps": int(rz.sum()),
+            "ms_resize_step_mean": float(t[rz].mean()) if rz.any() else None,
+            "ms_other_step_mean": float(t[~rz].mean()),
+            "capacity_steps_up": dbl, "capacity_steps_down": hlv,
+            "capacity": {"start": cap0, "max": max(caps), "end": caps[-1]}, "live_end": live,
+            "setup_s": {"generate": gen_s}}
 
 
 def batch_sweep(dev, batches=(100, 1_000, 10_000, 100_000, 1_000_000)):

@@ -417,6 +417,50 @@ __global__ void k_lvl_count(Lvl a, const uint32_t *__restrict__ cnt) {
   }
 }
 
+// High levels (few, huge windows): the window counts with every SM busy -- CTA (c, w) sums
+// chunk c of window w's leaf counts into nw[w] (zeroed first); k_lvl_accept then applies the
+// density test (Alg. 4 l.23-25, R5).  One CTA per window (k_lvl_count<TB>) left a 2^23-leaf
+// root window to a single SM: 8.4 of a 34 ms resizing batch.
+__global__ void __launch_bounds__(TB) k_lvl_count_wide(Lvl a, const uint32_t *__restrict__ cnt,
+                                                        uint32_t chunk_leaves) {
+  __shared__ uint64_t red[TB / 32];
+  const uint32_t q = a.widx[a.p];
+  const uint64_t w = blockIdx.y;
+  if (w >= q) return;
+  const uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+  const uint64_t c0 = (uint64_t)blockIdx.x * chunk_leaves;
+  uint64_t n = 0;
+  for (uint64_t l = c0 + threadIdx.x; l < c0 + chunk_leaves; l += TB) n += __ldg(cnt + leaf0 + l);
+  for (int o = 16; o; o >>= 1) n += __shfl_xor_sync(0xffffffffu, n, o);
+  if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = n;
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    uint64_t t = 0;
+    for (int k = 0; k < TB / 32; ++k) t += red[k];
+    if (t) atomicAdd((unsigned long long *)(a.nw + w), (unsigned long long)t);
+  }
+}
+
+__global__ void k_lvl_accept(Lvl a) {
+  const uint32_t q = a.widx[a.p];
+  for (uint64_t w = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; w < a.p;
+       w += (uint64_t)gridDim.x * blockDim.x) {
+    if (w >= q) {
+      a.acc[w] = 0;
+      a.nw[w] = 0;
+      continue;
+    }
+    const uint64_t n = a.nw[w];
+    const uint64_t u = a.wfirst[w + 1] - a.wfirst[w];
+    bool ok;
+    if (a.force) ok = true;
+    else if (a.op == GPMA_INSERT) ok = n + u <= a.tmax;
+    else ok = n >= u && n - u >= a.tmin;
+    a.acc[w] = ok ? 1u : 0u;
+    a.nw[w] = ok ? (a.op == GPMA_INSERT ? n + u : n - u) : 0;
+  }
+}
+
 __global__ void k_lvl_alist(Lvl a) {
   for (uint64_t w = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; w < a.p;
        w += (uint64_t)gridDim.x * blockDim.x)
@@ -457,27 +501,30 @@ __global__ void k_lvl_gather(Lvl a, const uint64_t *__restrict__ key, const uint
                              uint64_t bound_r) {
   const uint32_t nacc = a.aidx[a.p];
   const uint64_t wslots = (uint64_t)a.L << a.lvl;
+  const uint32_t lgw = (uint32_t)(__ffs(a.L) - 1) + a.lvl;        // wslots is a power of two
   const int lane = threadIdx.x & 31;
   const uint32_t lt = (1u << lane) - 1u;
   const uint32_t leafmask = (a.L == 32 ? 0xffffffffu : ((1u << a.L) - 1u) << (lane & ~(a.L - 1)));
-  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < bound_r;
+  // only the accepted windows' slots (rounded to whole warps: the ballot below needs them)
+  const uint64_t lim = min((uint64_t)bound_r, (uint64_t)((((uint64_t)nacc << lgw) + 31) & ~(uint64_t)31));
+  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < lim;
        g += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t ai = g / wslots;
+    uint64_t ai = g >> lgw;
     bool valid = ai < nacc;
     uint64_t k = KEY_NONE, s = 0;
     uint32_t v = 0, w = 0;
     if (valid) {
       w = a.alist[ai];
       uint64_t seg = a.pt[a.wfirst[w]] >> a.lvl;
-      s = seg * wslots + (g % wslots);
+      s = seg * wslots + (g & (wslots - 1));
       k = key[s];
       v = val[s];
     }
     bool live = valid && k != KEY_NONE && v != VAL_TOMB;
     uint32_t bal = __ballot_sync(0xffffffffu, live);
     if (live) {
-      uint64_t off = g % wslots;
-      uint64_t lidx = off / a.L;
+      uint64_t off = g & (wslots - 1);
+      uint64_t lidx = leaf_div(off, a.L);
       uint64_t rl = __popc(bal & leafmask & lt);
       if (a.lvl) rl += a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl];
       uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
@@ -533,15 +580,17 @@ __global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *
   const uint32_t nacc = a.aidx[a.p];
   const uint64_t Lc = 1ull << a.lvl;
   const uint64_t wslots = (uint64_t)a.L << a.lvl;
-  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < bound;
+  const uint32_t lgw = (uint32_t)(__ffs(a.L) - 1) + a.lvl;        // wslots is a power of two
+  const uint64_t lim = min(bound, (uint64_t)nacc << lgw);         // the accepted windows' slots only
+  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < lim;
        g += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t ai = g / wslots;
+    uint64_t ai = g >> lgw;
     if (ai >= nacc) continue;
     uint32_t w = a.alist[ai];
     uint64_t N = a.nw[w];
     uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
-    uint64_t off = g % wslots;
-    uint64_t l = off / a.L, p = off % a.L;
+    uint64_t off = g & (wslots - 1);
+    uint64_t l = leaf_div(off, a.L), p = leaf_mod(off, a.L);
     uint64_t lo = l * N / Lc, hi = (l + 1) * N / Lc;
     uint64_t s = leaf0 * a.L + off;
     if (p < hi - lo) {
@@ -957,7 +1006,14 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   GP_LAUNCH(g, k_lvl_first, gp, TB, 0, s, a);
   if (a.lvl <= 4) GP_LAUNCH(g, k_lvl_count<1>, grid_for(p), TB, 0, s, a, g->cnt);
   else if (a.lvl <= 11) GP_LAUNCH(g, k_lvl_count<32>, grid_for(p * 32), TB, 0, s, a, g->cnt);
-  else GP_LAUNCH(g, k_lvl_count<TB>, (unsigned)std::min<uint64_t>(p, MAX_RESIDENT_BLOCKS), TB, 0, s, a, g->cnt);
+  else {
+    const uint64_t nleaf_w = 1ull << a.lvl;
+    const uint32_t chunk = (uint32_t)std::min<uint64_t>(nleaf_w, 16384);
+    GP_CHECK(g, fill_zero(g, a.nw, p * 8, s));
+    GP_LAUNCH(g, k_lvl_count_wide, dim3((unsigned)(nleaf_w / chunk), (unsigned)wins_bound), TB, 0, s, a, g->cnt,
+              chunk);
+    GP_LAUNCH(g, k_lvl_accept, gp, TB, 0, s, a);
+  }
   scan_u32(g, a.acc, a.aidx, p, s);
   scan_u64(g, a.nw, a.woff, p, s);
   GP_LAUNCH(g, k_lvl_alist, gp, TB, 0, s, a);
