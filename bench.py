@@ -293,7 +293,9 @@ def run_gpma(args, rank, world, lrank):
                 h2d = B * (8 + 8 + 4)
                 d2h = 4 * V + 4 * V + 8 * V + ((8 * (V + 1) + 8 * nnz_e) if copy_csr else 0)
                 return {"value": 2 * B * args.e2e_steps * world / (ms_e2e / 1e3), "unit": "edge updates/s",
-                        "ms_per_step": ms_e2e / args.e2e_steps, "h2d_bytes_per_step": h2d,
+                        "ms_per_step": ms_e2e / args.e2e_steps,
+                        "ms_per_step_events": e0.elapsed_time(e1) / args.e2e_steps,
+                        "ms_per_step_wall": wall * 1e3 / args.e2e_steps, "h2d_bytes_per_step": h2d,
                         "d2h_bytes_per_step": d2h, "pr_iters": list(pipe.pr_iters)}
 
             # headline: every slide's batches H2D and its analytics results (BFS levels, CC
