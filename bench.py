@@ -468,6 +468,7 @@ def batch_sweep(dev, batches=(100, 1_000, 10_000, 100_000, 1_000_000)):
     cfg = CONFIGS[1]
     sw = config_stream(1, device=dev)
     res = []
+    analytics = None
     s = torch.cuda.Stream(dev)
     avail = sw.keys.numel() - sw.window
     with torch.cuda.stream(s):
@@ -495,6 +496,8 @@ def batch_sweep(dev, batches=(100, 1_000, 10_000, 100_000, 1_000_000)):
                         times.append(e0.elapsed_time(e1))
                         if alg == 1:
                             rounds.append(g.gpma_stats()["last_rounds"])
+                if alg == 0 and B == batches[-1]:
+                    analytics = _analytics_ms(g, cfg.V, sw, s)
                 del g
                 t = np.array(times)
                 point[name] = {"slides": len(times), "updates_per_s": 2 * B / (t.mean() / 1e3),
@@ -504,7 +507,38 @@ def batch_sweep(dev, batches=(100, 1_000, 10_000, 100_000, 1_000_000)):
                     point[name]["rounds_mean"] = float(np.mean(rounds))
             point["gpma_plus_speedup"] = point["gpma_plus"]["updates_per_s"] / point["gpma"]["updates_per_s"]
             res.append(point)
-    return {"workload": "configs[1] pokec-shaped (V=1.6M, 15M-edge window)", "points": res}
+    return {"workload": "configs[1] pokec-shaped (V=1.6M, 15M-edge window)", "points": res,
+            "analytics_after_update_ms": analytics}
+
+
+def _analytics_ms(g, V, sw, s):
+    """BFS / CC / PageRank (fp64, warm, tol 1e-3) / export on the updated configs[1] store
+    ("BFS/PR after the last slides"), mean of 3 runs each, CUDA events."""
+    dev = sw.keys.device
+    lv = torch.empty(V, dtype=torch.int32, device=dev)
+    lab = torch.empty(V, dtype=torch.int32, device=dev)
+    x = torch.empty(V, dtype=torch.float64, device=dev)
+    g.gpma_pagerank(x, warm_start=False, tol_l1=1e-3, max_iter=100, stream=s)
+    nnz = g.gpma_stats()["live_edges"]
+    rp = torch.empty(V + 1, dtype=torch.int64, device=dev)
+    col = torch.empty(nnz, dtype=torch.int32, device=dev)
+    cv = torch.empty(nnz, dtype=torch.int32, device=dev)
+    root = bfs_root(sw, CONFIGS[1].seed, 0)
+    jobs = {"bfs": lambda: g.gpma_bfs(root, lv, stream=s), "cc": lambda: g.gpma_cc(lab, stream=s),
+            "pagerank": lambda: g.gpma_pagerank(x, warm_start=True, tol_l1=1e-3, max_iter=100, stream=s),
+            "export_csr": lambda: g.gpma_export_csr(rp, col, cv, stream=s)}
+    out = {}
+    for name, fn in jobs.items():
+        ts = []
+        for _ in range(3):
+            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(s)
+            fn()
+            b.record(s)
+            b.synchronize()
+            ts.append(a.elapsed_time(b))
+        out[name] = float(np.mean(ts))
+    return out
 
 
 # ------------------------------------------------------------------ GPMA arm, N > 1
