@@ -91,3 +91,44 @@ def test_world_size_one_path():
     q = queue.Queue()
     _run(0, 1, 0, 0, 9, q)
     assert q.empty()
+
+
+def test_exchange_primitives_against_their_definitions():
+    """gpma_bfs_bits / gpma_bfs_merge / gpma_pr_update_rows (include/gpma.h) on a shard handle,
+    element by element against their plain definitions."""
+    from paper_journals_pvldb_shalht17_b200 import Gpma
+    from tests.gpu_helpers import DEV, keys_t, vals_t
+    V, P, r = 1000, 3, 1                                  # ragged: V not a multiple of 32 or P
+    chunk = (V + P - 1) // P
+    lo, hi = r * chunk, min(V, (r + 1) * chunk)
+    rng = np.random.default_rng(9)
+    src = rng.integers(lo, hi, 3000, dtype=np.uint64)
+    dst = rng.integers(0, V, 3000, dtype=np.uint64)
+    keys = np.unique((src << np.uint64(32)) | dst)
+    g = Gpma.gpma_create(V, keys_t(keys), vals_t(np.zeros(keys.size, np.uint32)), rows=(lo, hi))
+    words = (V + 31) // 32
+    # bits: levels == depth
+    lv = rng.integers(-1, 4, V).astype(np.int32)
+    bm = torch.zeros(words, dtype=torch.int32, device=DEV)
+    g.gpma_bfs_bits(torch.from_numpy(lv).to(DEV), 2, bm)
+    want = np.packbits(np.concatenate([lv == 2, np.zeros(words * 32 - V, bool)]), bitorder="little")
+    assert np.array_equal(bm.cpu().numpy().view(np.uint8), want)
+    # merge: unreached and set in any bitmap -> depth
+    bms = rng.integers(0, 1 << 32, (P, words), dtype=np.uint64).astype(np.uint32)
+    lvt = torch.from_numpy(lv).to(DEV)
+    g.gpma_bfs_merge(lvt, torch.from_numpy(bms.view(np.int32)).to(DEV), P, 7)
+    anyb = np.unpackbits(np.bitwise_or.reduce(bms, axis=0).view(np.uint8), bitorder="little")[:V].astype(bool)
+    exp = lv.copy()
+    exp[anyb & (lv == -1)] = 7
+    assert np.array_equal(lvt.cpu().numpy(), exp)
+    # owned-rows PageRank update from reduced sums (2^-62 fixed point) + the dangling total
+    S = float(2 ** 62)
+    x = rng.random(V)
+    yr = rng.integers(0, 1 << 50, hi - lo + 1, dtype=np.uint64)
+    xt = torch.from_numpy(x.copy()).to(DEV)
+    err = g.gpma_pr_update_rows(xt, torch.from_numpy(yr.view(np.int64)).to(DEV), 0.85)
+    nx = (1 - 0.85) / V + 0.85 * (yr[:-1].astype(np.float64) / S + float(yr[-1]) / S / V)
+    got = xt.cpu().numpy()
+    assert np.abs(got[lo:hi] - nx).max() <= 1e-15
+    assert np.array_equal(got[:lo], x[:lo]) and np.array_equal(got[hi:], x[hi:])
+    assert abs(err - np.abs(nx - x[lo:hi]).sum()) <= 1e-9
