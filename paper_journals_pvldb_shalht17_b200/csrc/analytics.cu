@@ -977,7 +977,8 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   int queued = 0, cur = 0;
   uint32_t it = 0;
   while (queued < max_iter) {
-    const int batch = std::min(queued == 0 ? 2 : 1, max_iter - queued);
+    // (tol <= 0 never stops early -- the fixed-K parity mode, R20: queue every iteration at once)
+    const int batch = tol <= 0.0 ? max_iter - queued : std::min(queued == 0 ? 2 : 1, max_iter - queued);
     for (int b = 0; b < batch; ++b, ++queued) {
       GP_LAUNCH(g, k_pr_iter_begin, 1, 32, 0, s, acc, cur ^ 1, lp);
       // destination passes: random REDs run ~3x faster while their target fits in L2
