@@ -622,6 +622,144 @@ __global__ void k_lvl_keep(Lvl a) {
   }
 }
 
+// ---- small levels (p <= 4096 pending, windows of <= 64 leaves): one CTA runs the
+// segment / count / accept front (UniqueSegments, CountSegment, density test, the accepted
+// list: 7 launches) and another the keep / compaction-offset / summary back (3 launches).
+// Above level 0 the pending lists are small and every launch is a few us of pure overhead.
+constexpr int LS_T = 1024, LS_I = 4;
+constexpr uint64_t LS_MAXP = (uint64_t)LS_T * LS_I;
+constexpr uint32_t LS_MAXLVL = 4;                     // windows of <= 16 leaves: counted in-thread
+
+// exclusive scan of 4 consecutive items per thread over the CTA; returns the total
+__device__ __forceinline__ uint64_t ls_scan4(uint64_t v[LS_I], uint64_t *wsum) {
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  uint64_t ex[LS_I];
+  uint64_t t = 0;
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i) {
+    ex[i] = t;
+    t += v[i];
+  }
+  uint64_t x = t;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint64_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if (lane >= o) x += y;
+  }
+  if (lane == 31) wsum[warp] = x;
+  __syncthreads();
+  if (warp == 0) {
+    uint64_t w = wsum[lane];
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint64_t y = __shfl_up_sync(0xffffffffu, w, o);
+      if (lane >= o) w += y;
+    }
+    wsum[lane] = w;
+  }
+  __syncthreads();
+  const uint64_t base = (warp ? wsum[warp - 1] : 0) + x - t;
+  const uint64_t total = wsum[31];
+  __syncthreads();                                     // wsum is reused by the next scan
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i) v[i] = base + ex[i];
+  return total;
+}
+
+__global__ void __launch_bounds__(LS_T) k_lvl_front_small(Lvl a, const uint32_t *__restrict__ cnt) {
+  __shared__ uint64_t wsum[32];
+  const uint64_t p = a.p;
+  const uint64_t j0 = (uint64_t)threadIdx.x * LS_I;
+  uint64_t f[LS_I];
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i) {                     // window-head flags (l.18-21: RLE)
+    const uint64_t j = j0 + i;
+    f[i] = (j < p && (j == 0 || (a.pt[j] >> a.lvl) != (a.pt[j - 1] >> a.lvl))) ? 1u : 0u;
+    if (j < p) a.hf[j] = (uint32_t)f[i];
+  }
+  uint64_t e[LS_I] = {f[0], f[1], f[2], f[3]};
+  const uint64_t q = ls_scan4(e, wsum);                // windows
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i) {
+    const uint64_t j = j0 + i;
+    if (j < p) {
+      a.widx[j] = (uint32_t)e[i];
+      if (f[i]) a.wfirst[e[i]] = (uint32_t)j;
+    }
+  }
+  if (threadIdx.x == 0) {
+    a.widx[p] = (uint32_t)q;
+    a.wfirst[q] = (uint32_t)p;
+  }
+  __syncthreads();
+  uint64_t ac[LS_I], nw[LS_I];
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i) {                     // count + density test (l.23-25, R5)
+    const uint64_t w = j0 + i;
+    ac[i] = nw[i] = 0;
+    if (w < q) {
+      const uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+      uint64_t n = 0;
+#pragma unroll
+      for (uint32_t l = 0; l < (1u << LS_MAXLVL); ++l)   // independent loads, all in flight
+        if (l < (1u << a.lvl)) n += cnt[leaf0 + l];
+      const uint64_t u = a.wfirst[w + 1] - a.wfirst[w];
+      bool ok;
+      if (a.force) ok = true;
+      else if (a.op == GPMA_INSERT) ok = n + u <= a.tmax;
+      else ok = n >= u && n - u >= a.tmin;
+      ac[i] = ok ? 1u : 0u;
+      nw[i] = ok ? (a.op == GPMA_INSERT ? n + u : n - u) : 0;
+    }
+    if (w < p) {
+      a.acc[w] = (uint32_t)ac[i];
+      a.nw[w] = nw[i];
+    }
+  }
+  uint64_t ai[LS_I] = {ac[0], ac[1], ac[2], ac[3]};
+  const uint64_t nacc = ls_scan4(ai, wsum);
+  const uint64_t tot = ls_scan4(nw, wsum);
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i) {
+    const uint64_t w = j0 + i;
+    if (w < p) {
+      a.aidx[w] = (uint32_t)ai[i];
+      a.woff[w] = nw[i];
+      if (ac[i]) a.alist[ai[i]] = (uint32_t)w;
+    }
+  }
+  if (threadIdx.x == 0) {
+    a.aidx[p] = (uint32_t)nacc;
+    a.woff[p] = tot;
+  }
+}
+
+__global__ void __launch_bounds__(LS_T) k_lvl_back_small(Lvl a, Ctrl *c) {
+  __shared__ uint64_t wsum[32];
+  const uint64_t p = a.p;
+  const uint64_t j0 = (uint64_t)threadIdx.x * LS_I;
+  uint64_t k[LS_I];
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i) {                     // promote the rejected (l.12-15)
+    const uint64_t j = j0 + i;
+    k[i] = 0;
+    if (j < p) {
+      const uint32_t w = a.widx[j] + a.hf[j] - 1;
+      k[i] = a.acc[w] ? 0u : 1u;
+      a.keep[j] = (uint32_t)k[i];
+    }
+  }
+  const uint64_t tot = ls_scan4(k, wsum);
+#pragma unroll
+  for (int i = 0; i < LS_I; ++i)
+    if (j0 + i < p) a.kpos[j0 + i] = (uint32_t)k[i];
+  if (threadIdx.x == 0) {
+    a.kpos[p] = (uint32_t)tot;
+    c->sum = (uint64_t)a.widx[p] | ((uint64_t)a.aidx[p] << 32);
+    c->sum2 = tot;
+  }
+}
+
 __global__ void k_lvl_summary(Lvl a, Ctrl *c) {
   // sum  = unique windows | accepted windows << 32 ; sum2 = pending after this level
   c->sum = (uint64_t)a.widx[a.p] | ((uint64_t)a.aidx[a.p] << 32);
@@ -993,6 +1131,12 @@ struct LevelOut {
   uint64_t q, nacc, p_new;
 };
 
+// single-CTA front / back of small levels (GPMA_LVL_SMALL=0 disables; read per call)
+static bool lvl_small_on() {
+  const char *e = getenv("GPMA_LVL_SMALL");
+  return !e || atoi(e) != 0;
+}
+
 static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t *dirty_base,
                               cudaStream_t s, bool resize_target, uint64_t new_cap, uint64_t *nk,
                               uint32_t *nv, uint32_t *ncnt) {
@@ -1001,6 +1145,10 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   const uint64_t wins_bound = std::min<uint64_t>(p, nleaves >> a.lvl);
   const uint64_t wslots = (uint64_t)g->L << a.lvl;
   const unsigned gp = grid_for(p);
+  const bool small = p <= LS_MAXP && a.lvl <= LS_MAXLVL && lvl_small_on();
+  if (small) {
+    GP_LAUNCH(g, k_lvl_front_small, 1, LS_T, 0, s, a, g->cnt);
+  } else {
   GP_LAUNCH(g, k_lvl_flags, gp, TB, 0, s, a);
   scan_u32(g, a.hf, a.widx, p, s);
   GP_LAUNCH(g, k_lvl_first, gp, TB, 0, s, a);
@@ -1017,6 +1165,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   scan_u32(g, a.acc, a.aidx, p, s);
   scan_u64(g, a.nw, a.woff, p, s);
   GP_LAUNCH(g, k_lvl_alist, gp, TB, 0, s, a);
+  }
   // scratch: sum of merged window sizes <= wins_bound * wslots (and <= cap + p)
   uint64_t need = a.force ? g->cap + p : wins_bound * wslots;
   GP_CHECK(g, ensure(g->b_wk, need * 8, s));
@@ -1047,9 +1196,13 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     GP_LAUNCH(g, k_layout_even, grid_for(new_cap), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
               g->row_offset, g->L, nl_new, g->rb);
   }
-  GP_LAUNCH(g, k_lvl_keep, gp, TB, 0, s, a);
-  scan_u32(g, a.keep, a.kpos, p, s);
-  GP_LAUNCH(g, k_lvl_summary, 1, 1, 0, s, a, g->ctrl_d);
+  if (small) {
+    GP_LAUNCH(g, k_lvl_back_small, 1, LS_T, 0, s, a, g->ctrl_d);
+  } else {
+    GP_LAUNCH(g, k_lvl_keep, gp, TB, 0, s, a);
+    scan_u32(g, a.keep, a.kpos, p, s);
+    GP_LAUNCH(g, k_lvl_summary, 1, 1, 0, s, a, g->ctrl_d);
+  }
   if (g->trace_on) {
     // copy segment starts / offsets / flags of this level (debug only)
     std::vector<uint32_t> wf(p + 1), ac(p + 1), pt(p), wi(p + 1);
