@@ -350,6 +350,7 @@ struct Lvl {
   int force;           // resize: accept the single root window unconditionally
   uint32_t rb;         // first owned row (row offsets are local)
   uint64_t nleaves;    // leaves of the store (offset of the guard counts after the masks)
+  const uint32_t *lcnt; // small levels: leaf live counts read directly instead of the prefix lpre
 };
 
 __global__ void k_lvl_flags(Lvl a) {
@@ -526,7 +527,14 @@ __global__ void k_lvl_gather(Lvl a, const uint64_t *__restrict__ key, const uint
       uint64_t off = g & (wslots - 1);
       uint64_t lidx = leaf_div(off, a.L);
       uint64_t rl = __popc(bal & leafmask & lt);
-      if (a.lvl) rl += a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl];
+      if (a.lvl) {
+        if (a.lcnt) {                                  // <= 15 earlier leaves of a small window
+          const uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+          for (uint64_t l = 0; l < lidx; ++l) rl += a.lcnt[leaf0 + l];
+        } else {
+          rl += a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl];
+        }
+      }
       uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
       uint64_t c = lower_bound_u64(a.pk, ub, ue, k) - ub;
       uint64_t r;
@@ -557,7 +565,14 @@ __global__ void k_lvl_place(Lvl a, const uint64_t *__restrict__ key, const uint3
     uint64_t k = a.pk[j];
     uint64_t seg = t >> a.lvl;
     uint64_t lidx = t - (seg << a.lvl);
-    uint64_t rl = a.lvl ? a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl] : 0;
+    uint64_t rl = 0;
+    if (a.lvl) {
+      if (a.lcnt) {                                    // small window: sum the earlier leaves
+        for (uint64_t l = 0; l < lidx; ++l) rl += a.lcnt[(seg << a.lvl) + l];
+      } else {
+        rl = a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl];
+      }
+    }
     uint64_t base = (uint64_t)t * a.L;
     for (uint32_t p = 0; p < a.L; ++p) {
       uint64_t x = key[base + p];
@@ -1172,7 +1187,10 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   GP_CHECK(g, ensure(g->b_wv, need * 4, s));
   a.wk = (uint64_t *)g->b_wk.p;
   a.wv = (uint32_t *)g->b_wv.p;
-  if (a.lvl) {
+  a.lcnt = nullptr;
+  if (small && a.lvl) {
+    a.lcnt = g->cnt;                                   // the gather sums its window's leaves itself
+  } else if (a.lvl) {
     uint64_t lb = wins_bound << a.lvl;
     GP_CHECK(g, ensure(g->b_lpre, (lb + 1) * 8, s));
     a.lpre = (uint64_t *)g->b_lpre.p;
