@@ -2,7 +2,7 @@
 # compute-sanitizer over representative GPU parity tests (run under gpurun, 1 GPU)
 mkdir -p gpurun_out
 SEL='config0_sliding_window_lazy[0] or config0_sliding_window_rebalance[0] or random_small_with_resizes[0-1] or random_small_with_resizes[1-0] or gpma_lock_example2 or example4'
-SEL2='graph_replayed_sliding_window[0-0] or graph_replayed_sliding_window[0-1] or replay_errors or across_resizes[0-0] or every_strategy[10] or every_sample_strategy[10]'
+SEL2='graph_replayed_sliding_window[0-0] or graph_replayed_sliding_window[0-1] or replay_errors or across_resizes[0-0] or every_strategy[10] or every_sample_strategy[10] or level_step_paths'
 for tool in memcheck racecheck synccheck; do
   compute-sanitizer --tool $tool --error-exitcode 9 --print-limit 20 \
     python -m pytest tests/test_gpu_parity.py tests/test_gpu_query.py tests/test_gpu_edge_cases.py \
