@@ -629,6 +629,107 @@ __global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *
   }
 }
 
+// Small levels (windows of <= 16 leaves, <= 512 slots): gather + placement + even
+// re-dispatch of one accepted window in one CTA, the merged list staged in shared memory
+// instead of the HBM scratch (Alg. 4 l.26-27, R7) -- the three kernels above fused.
+constexpr int LM_T = 256, LM_MAXS = 512;
+__global__ void __launch_bounds__(LM_T) k_lvl_merge_small(Lvl a, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
+                                                          uint32_t *__restrict__ cnt, uint32_t *__restrict__ tmask,
+                                                          uint64_t *__restrict__ row_offset, uint2 *__restrict__ dirty,
+                                                          uint64_t dirty_base) {
+  __shared__ uint64_t mk[LM_MAXS];
+  __shared__ uint32_t mv[LM_MAXS];
+  __shared__ uint32_t lpre[17];
+  const uint32_t nacc = a.aidx[a.p];
+  const uint32_t ai = blockIdx.x;
+  if (ai >= nacc) return;                              // uniform: the whole CTA leaves
+  const uint32_t w = a.alist[ai];
+  const uint32_t Lc = 1u << a.lvl;
+  const uint32_t ws = a.L << a.lvl;
+  const uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+  const uint64_t N = a.nw[w];
+  const uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint32_t leafmask = (a.L == 32 ? 0xffffffffu : ((1u << a.L) - 1u) << (lane & ~(a.L - 1)));
+  if (threadIdx.x == 0) {                              // live entries before each leaf
+    uint32_t acc = 0;
+    for (uint32_t l = 0; l < Lc; ++l) {
+      lpre[l] = acc;
+      acc += cnt[leaf0 + l];
+    }
+    lpre[Lc] = acc;
+  }
+  __syncthreads();
+  for (uint32_t o0 = 0; o0 < ws; o0 += LM_T) {         // gather the live entries (whole warps)
+    const uint32_t off = o0 + threadIdx.x;
+    const bool in = off < ws;
+    uint64_t k = KEY_NONE;
+    uint32_t v = 0;
+    if (in) {
+      k = key[leaf0 * a.L + off];
+      v = val[leaf0 * a.L + off];
+    }
+    const bool live = in && k != KEY_NONE && v != VAL_TOMB;
+    const uint32_t bal = __ballot_sync(0xffffffffu, live);
+    if (live) {
+      const uint64_t rl = __popc(bal & leafmask & lt) + lpre[leaf_div(off, a.L)];
+      const uint64_t c = lower_bound_u64(a.pk, ub, ue, k) - ub;
+      bool drop = false;
+      uint64_t r;
+      if (a.op == GPMA_INSERT) {
+        r = rl + c;
+      } else {
+        drop = (ub + c < ue) && a.pk[ub + c] == k;
+        r = rl - c;
+      }
+      if (!drop) {
+        mk[r] = k;
+        mv[r] = v;
+      }
+    }
+  }
+  if (a.op == GPMA_INSERT) {                           // place the window's insertions
+    for (uint64_t j = ub + threadIdx.x; j < ue; j += LM_T) {
+      const uint64_t k = a.pk[j];
+      const uint32_t t = a.pt[j];
+      uint64_t rl = lpre[t - leaf0];
+      const uint64_t base = (uint64_t)t * a.L;
+      for (uint32_t q = 0; q < a.L; ++q) {
+        const uint64_t x = key[base + q];
+        if (x == KEY_NONE || x > k) break;
+        if (val[base + q] != VAL_TOMB) ++rl;
+      }
+      const uint64_t r = (j - ub) + rl;
+      mk[r] = k;
+      mv[r] = a.pv[j];
+    }
+  }
+  __syncthreads();                                     // every read of the window is done
+  for (uint32_t off = threadIdx.x; off < ws; off += LM_T) {   // re-dispatch evenly (R7)
+    const uint64_t l = leaf_div(off, a.L), q = leaf_mod(off, a.L);
+    const uint64_t lo = l * N / Lc, hi = (l + 1) * N / Lc;
+    const uint64_t sl = leaf0 * a.L + off;
+    if (q < hi - lo) {
+      const uint64_t k = mk[lo + q];
+      key[sl] = k;
+      val[sl] = mv[lo + q];
+      if (is_guard_key(k)) row_offset[(k >> 32) - a.rb + 1] = sl;
+    } else {
+      key[sl] = KEY_NONE;
+      val[sl] = 0;
+    }
+    if (q == 0) {
+      cnt[leaf0 + l] = (uint32_t)(hi - lo);
+      tmask[leaf0 + l] = 0u;                          // tombstones are dropped by a rewrite
+      uint32_t gc = 0;
+      for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(mk[e]);
+      tmask[a.nleaves + leaf0 + l] = gc;              // guards per leaf (third section)
+    }
+  }
+  if (threadIdx.x == 0) dirty[dirty_base + ai] = make_uint2((uint32_t)leaf0, Lc);
+}
+
 __global__ void k_lvl_keep(Lvl a) {
   for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < a.p;
        j += (uint64_t)gridDim.x * blockDim.x) {
@@ -1147,9 +1248,9 @@ struct LevelOut {
 };
 
 // single-CTA front / back of small levels (GPMA_LVL_SMALL=0 disables; read per call)
-static bool lvl_small_on() {
+static int lvl_small_on() {      // 0 off, 1 front/back only, 2 (default) + fused window merge
   const char *e = getenv("GPMA_LVL_SMALL");
-  return !e || atoi(e) != 0;
+  return e ? atoi(e) : 2;
 }
 
 static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t *dirty_base,
@@ -1181,38 +1282,44 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   scan_u64(g, a.nw, a.woff, p, s);
   GP_LAUNCH(g, k_lvl_alist, gp, TB, 0, s, a);
   }
-  // scratch: sum of merged window sizes <= wins_bound * wslots (and <= cap + p)
-  uint64_t need = a.force ? g->cap + p : wins_bound * wslots;
-  GP_CHECK(g, ensure(g->b_wk, need * 8, s));
-  GP_CHECK(g, ensure(g->b_wv, need * 4, s));
-  a.wk = (uint64_t *)g->b_wk.p;
-  a.wv = (uint32_t *)g->b_wv.p;
-  a.lcnt = nullptr;
-  if (small && a.lvl) {
-    a.lcnt = g->cnt;                                   // the gather sums its window's leaves itself
-  } else if (a.lvl) {
-    uint64_t lb = wins_bound << a.lvl;
-    GP_CHECK(g, ensure(g->b_lpre, (lb + 1) * 8, s));
-    a.lpre = (uint64_t *)g->b_lpre.p;
-    GP_LAUNCH(g, k_lvl_leafcnt, grid_for(lb), TB, 0, s, a, g->cnt, lb);
-    scan_u64(g, a.lpre, a.lpre, lb, s);
-  }
-  uint64_t bslots = wins_bound * wslots;
-  uint64_t bslots_r = (bslots + 31) & ~31ull;
-  GP_LAUNCH(g, k_lvl_gather, grid_for(bslots_r), TB, 0, s, a, g->key, g->val, bslots_r);
-  if (a.op == GPMA_INSERT) GP_LAUNCH(g, k_lvl_place, gp, TB, 0, s, a, g->key, g->val);
-  if (!resize_target) {
-    GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots), TB, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
-              g->row_offset, bslots, (uint2 *)g->b_dirty.p, *dirty_base);
+  const bool merge_small = small && !resize_target && wslots <= (uint64_t)LM_MAXS && lvl_small_on() > 1;
+  if (merge_small) {
+    GP_LAUNCH(g, k_lvl_merge_small, (unsigned)wins_bound, LM_T, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
+              g->row_offset, (uint2 *)g->b_dirty.p, *dirty_base);
   } else {
-    // the single root window, laid out over the whole new array
-    uint64_t N;
-    GP_CHECK(g, readback(g, &g->ctrl_h->sum, a.nw, 8, s));
-    GP_CHECK(g, cudaStreamSynchronize(s));
-    N = g->ctrl_h->sum;
-    uint64_t nl_new = new_cap / g->L;
-    GP_LAUNCH(g, k_layout_even, grid_for(new_cap), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
-              g->row_offset, g->L, nl_new, g->rb);
+    // scratch: sum of merged window sizes <= wins_bound * wslots (and <= cap + p)
+    uint64_t need = a.force ? g->cap + p : wins_bound * wslots;
+    GP_CHECK(g, ensure(g->b_wk, need * 8, s));
+    GP_CHECK(g, ensure(g->b_wv, need * 4, s));
+    a.wk = (uint64_t *)g->b_wk.p;
+    a.wv = (uint32_t *)g->b_wv.p;
+    a.lcnt = nullptr;
+    if (small && a.lvl) {
+      a.lcnt = g->cnt;                                   // the gather sums its window's leaves itself
+    } else if (a.lvl) {
+      uint64_t lb = wins_bound << a.lvl;
+      GP_CHECK(g, ensure(g->b_lpre, (lb + 1) * 8, s));
+      a.lpre = (uint64_t *)g->b_lpre.p;
+      GP_LAUNCH(g, k_lvl_leafcnt, grid_for(lb), TB, 0, s, a, g->cnt, lb);
+      scan_u64(g, a.lpre, a.lpre, lb, s);
+    }
+    uint64_t bslots = wins_bound * wslots;
+    uint64_t bslots_r = (bslots + 31) & ~31ull;
+    GP_LAUNCH(g, k_lvl_gather, grid_for(bslots_r), TB, 0, s, a, g->key, g->val, bslots_r);
+    if (a.op == GPMA_INSERT) GP_LAUNCH(g, k_lvl_place, gp, TB, 0, s, a, g->key, g->val);
+    if (!resize_target) {
+      GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots), TB, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
+                g->row_offset, bslots, (uint2 *)g->b_dirty.p, *dirty_base);
+    } else {
+      // the single root window, laid out over the whole new array
+      uint64_t N;
+      GP_CHECK(g, readback(g, &g->ctrl_h->sum, a.nw, 8, s));
+      GP_CHECK(g, cudaStreamSynchronize(s));
+      N = g->ctrl_h->sum;
+      uint64_t nl_new = new_cap / g->L;
+      GP_LAUNCH(g, k_layout_even, grid_for(new_cap), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
+                g->row_offset, g->L, nl_new, g->rb);
+    }
   }
   if (small) {
     GP_LAUNCH(g, k_lvl_back_small, 1, LS_T, 0, s, a, g->ctrl_d);

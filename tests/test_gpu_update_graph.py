@@ -133,11 +133,12 @@ def test_graph_replay_across_resizes(seed, mode):
     assert_same_csr(g, o)
 
 
-@pytest.mark.parametrize("small", ["0", "1"])
+@pytest.mark.parametrize("small", ["0", "1", "2"])
 @pytest.mark.parametrize("mode", [0, 1])
 def test_level_step_paths(small, mode):
-    """Levels >= 1 through the single-CTA small-level front/back (GPMA_LVL_SMALL=1, default)
-    and through the multi-kernel step (0): layouts and per-level traces (segments, offsets,
+    """Levels >= 1 through the single-CTA small-level front/back with the fused per-window
+    merge (GPMA_LVL_SMALL=2, default), front/back only (1) and the multi-kernel step (0):
+    layouts and per-level traces (segments, offsets,
     flags of every round, Alg. 4 l.7-25) equal the oracle's on configs[0] sliding windows and
     on random batches that climb to the root and resize."""
     from tests.test_gpu_parity import _slide_parity, test_random_small_with_resizes
