@@ -457,6 +457,7 @@ def resize_stress(dev, grow_steps=242, shrink_steps=248):
             "updates_per_s": upd / (t.sum() / 1e3), "ms_per_step_mean": float(t.mean()),
             "steps": int(t.size), "resize_steps": int(rz.sum()),
             "ms_resize_step_mean": float(t[rz].mean()) if rz.any() else None,
+            "ms_resize_steps": [round(float(x), 3) for x in t[rz]],
             "ms_other_step_mean": float(t[~rz].mean()),
             "capacity_steps_up": dbl, "capacity_steps_down": hlv,
             "capacity": {"start": cap0, "max": max(caps), "end": caps[-1]}, "live_end": live,
