@@ -16,10 +16,10 @@ namespace gp {
 cudaError_t ensure(DevBuf &b, size_t bytes, cudaStream_t s) {
   if (bytes == 0) bytes = 16;
   if (b.bytes >= bytes) return cudaSuccess;
+  const size_t want = std::max(bytes, b.bytes + b.bytes / 2);  // grow x1.5 at least
   if (b.p) cudaFreeAsync(b.p, s);
   b.p = nullptr;
   b.bytes = 0;
-  size_t want = std::max(bytes, (size_t)(b.bytes * 3 / 2));
   cudaError_t e = cudaMallocAsync(&b.p, want, s);
   if (e != cudaSuccess) {
     b.p = nullptr;
