@@ -75,7 +75,8 @@ typedef struct {
   uint16_t init_density_bp;   /* R15: 6000                                            */
   uint16_t algorithm;         /* insertion: 0 = GPMA+ segment-oriented (Alg. 4, default);
                                  1 = GPMA lock-based (Alg. 1) with deterministic
-                                 lock arbitration (the smallest key wins a segment)       */
+                                 lock arbitration (R28: the contender from the highest
+                                 child segment wins, then the smallest key; Ex. 2)      */
   uint32_t delete_mode;       /* gpma_delete_mode                                     */
   uint32_t row_begin, row_end;/* shard (R24): the store holds the rows
                                  (sources) [row_begin, row_end) only -- guards, row

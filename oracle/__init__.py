@@ -6,9 +6,11 @@ Only ``tests/``, ``__graft_entry__.smoke()`` and ``bench.py``'s ``cpu_baseline``
 
 The arithmetic lives in ``oracle/gpma_oracle.c`` (plain single-threaded C, -O2,
 no SIMD intrinsics); this module is a ctypes wrapper plus numpy marshalling.
-Each C function cites the PAPER.md passage it follows.  Parity unpinned (by
-the paper): the root resize rule (R6/R14) and the strict-delete layout -- those
-are checked by invariants and brute-force logical-set replay only.
+Each C function cites the PAPER.md passage it follows.  The root resize rule
+(R6/R14) and the strict-delete layout, which no printed example reaches, are
+pinned by hand-derived examples (tests/test_oracle_resize_pins.py) and
+minimality properties; tools/oracle_mutations.sh shows each pin catching a
+plausible mistake.
 """
 from __future__ import annotations
 
@@ -64,6 +66,7 @@ def lib():
             "orc_bfs_csr": (None, [u32, P, P, u32, P]),
             "orc_set_algorithm": (None, [P, i32]),
             "orc_rounds_last": (u64, [P]),
+            "orc_set_max_rounds": (None, [P, u64]),
             "orc_cc_csr": (None, [u32, P, P, P]),
             "orc_pagerank_csr": (i32, [u32, P, P, P, i32, C.c_double, C.c_double, i32]),
         }
@@ -145,6 +148,10 @@ class Oracle:
     def rounds(self) -> int:
         """GPMA (Alg. 1): retry rounds of the last insert batch."""
         return int(lib().orc_rounds_last(self._h))
+
+    def set_max_rounds(self, r: int):
+        """GPMA (Alg. 1) test hook: stop a batch after r rounds (0 = until every insertion took effect)."""
+        lib().orc_set_max_rounds(self._h, r)
 
     def __del__(self):
         if getattr(self, "_h", None):

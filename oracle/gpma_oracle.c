@@ -18,10 +18,13 @@
  * connected components and power-iteration PageRank
  * on the exported CSR.
  *
- * Readings of silent / garbled passages are SURVEY.md §8(c) R1-R27, repeated
- * in DESIGN.md "Readings".  Pins: tests/test_oracle_*.py.  Parity-unpinned
- * parts (self-consistency + invariants + brute-force logical set only): the
- * root-resize rule (R6, R14) and the strict-delete layout.
+ * Readings of silent / garbled passages are SURVEY.md §8(c) R1-R29, repeated
+ * in DESIGN.md "Readings".  Pins: tests/test_oracle_*.py -- the paper's worked
+ * examples (Fig. 3, Ex. 1, Ex. 2, Ex. 4, Fig. 5), hand-derived root-resize and
+ * strict-delete examples on the Fig. 3-size PMA (R6, R14, min_i;
+ * tests/test_oracle_resize_pins.py), brute-force replay, closed forms and
+ * library routines for the analytics; tools/oracle_mutations.sh checks that a
+ * plausible mistake in each rule fails a pin.
  */
 #include <stdint.h>
 #include <stdlib.h>
@@ -57,6 +60,7 @@ typedef struct orc {
   uint64_t resizes, resizes_last;
   int algorithm;       /* 0 = GPMA+ (Alg. 4), 1 = GPMA lock-based (Alg. 1)            */
   uint64_t rounds_last;/* GPMA: retry rounds of the last batch                        */
+  uint64_t max_rounds; /* GPMA test hook: stop after this many rounds (0 = until done) */
 } orc_t;
 
 /* ---------------------------------------------------------------- thresholds */
@@ -390,18 +394,22 @@ static int cmp_upd(const void *a, const void *b) {
  * arbitration: every insertion searches its leaf, then the rounds climb level by level
  * ("all threads are synchronized after updating all segments located at the same tree
  * height").  At each level the insertions that reach the same segment compete for
- * its lock; the one with the smallest key wins (the paper leaves the winner unspecified --
- * "Assuming Insertion-1 succeeds") and the others abort until the next round
- * (l.11-12).  A winner whose segment can take one more entry (count + 1 <= max_i, R5) merges
- * and re-dispatches it (l.16-17); otherwise it climbs (l.13-14).  As for GPMA+ (R6), the root
- * is tested too; a winner the root cannot take doubles it (l.20) and retries next round.  Rounds repeat until every insertion
- * took effect (l.2). */
+ * its lock and the others abort until the next round (l.11-12).  The paper leaves the winner
+ * open ("Assuming Insertion-1 succeeds"; "Insertion-48 wins"); R28: the
+ * contender that climbed from the highest child segment wins, and among contenders of one
+ * child (always the case at the leaves) the smallest key -- the one rule that reproduces both
+ * printed choices of Ex. 2 (1 beats 4 in leaf 0; 48 from leaf 7 beats 35 from leaf 6 for
+ * segment [24,31]).  A winner whose segment can take one more entry (count + 1 <= max_i, R5)
+ * merges and re-dispatches it (l.16-17); otherwise it climbs (l.13-14).  As for GPMA+ (R6),
+ * the root is tested too; a winner the root cannot take doubles it (l.20) and retries next
+ * round.  Rounds repeat until every insertion took effect (l.2), or -- test hook only --
+ * until max_rounds rounds ran (the aborted insertions are then dropped). */
 static int gpma_lock_insert(orc_t *o, upd_t *P, uint64_t np) {
   upd_t *A = (upd_t *)malloc(sizeof(upd_t) * (np ? np : 1));
   upd_t *W = (upd_t *)malloc(sizeof(upd_t) * (np ? np : 1));
   uint64_t *wk = NULL; uint32_t *wv = NULL; uint64_t wcap = 0;
   o->rounds_last = 0;
-  while (np > 0) {
+  while (np > 0 && (!o->max_rounds || o->rounds_last < o->max_rounds)) {
     uint64_t na = 0, nw, j, nne;
     uint32_t i;
     uint64_t *ne = nonempty_leaves(o, &nne);
@@ -413,8 +421,20 @@ static int gpma_lock_insert(orc_t *o, upd_t *P, uint64_t np) {
     for (i = 0; i <= o->h && nw > 0; i++) {           /* up to the root, tested too (R6) */
       uint64_t nk = 0, g0 = 0;
       while (g0 < nw) {
-        uint64_t seg = W[g0].leaf >> i, g1 = g0 + 1, s0, s1, n = 0, s;
-        while (g1 < nw && (W[g1].leaf >> i) == seg) A[na++] = W[g1++];   /* lose the lock: abort */
+        uint64_t seg = W[g0].leaf >> i, g1 = g0 + 1, s0, s1, n = 0, s, win, c;
+        while (g1 < nw && (W[g1].leaf >> i) == seg) g1++;  /* contenders W[g0..g1), by key */
+        /* R28: the highest child wins (child = leaf >> (i-1); one child at the leaves), and
+         * within it the smallest key: the first contender of the last child run */
+        win = g1 - 1;
+        if (i > 0) {
+          c = W[g1 - 1].leaf >> (i - 1);
+          while (win > g0 && (W[win - 1].leaf >> (i - 1)) == c) win--;
+        } else {
+          win = g0;
+        }
+        for (s = g0; s < g1; s++)
+          if (s != win) A[na++] = W[s];                 /* lose the lock: abort (l.11-12) */
+        W[g0] = W[win];                                 /* the winner goes on below      */
         s0 = (seg << i) * o->L; s1 = s0 + ((uint64_t)o->L << i);
         for (s = s0; s < s1; s++) n += is_live(o, s);
         if (n + 1 <= o->tmax[i]) {                    /* l.13 test fails -> insert (l.16-17) */
@@ -458,6 +478,7 @@ static int gpma_lock_insert(orc_t *o, upd_t *P, uint64_t np) {
 }
 
 void orc_set_algorithm(orc_t *o, int algorithm) { o->algorithm = algorithm; }
+void orc_set_max_rounds(orc_t *o, uint64_t r) { o->max_rounds = r; }
 uint64_t orc_rounds_last(const orc_t *o) { return o->rounds_last; }
 
 /* GpmaPlusInsertion (Alg. 4) and its dual for strict deletions over the

@@ -1480,8 +1480,38 @@ __global__ void k_relocate(const uint64_t *__restrict__ pk, uint64_t p, const ui
     pt[j] = locate_leaf(head, nleaves, pk[j]);
 }
 
-// lock arbitration at one level: the first (smallest key) insertion of every segment keeps
-// going (winner list), the others abort to the next round (loser list, appended at `na`)
+// Lock arbitration at level `lvl` (R28): among the insertions that reach one segment, the
+// contender that climbed from the highest child segment (child = leaf >> (lvl-1)) wins, and
+// among contenders of one child -- always the case at the leaves -- the smallest key: the
+// first contender of the segment's last child run (Ex. 2: 1 beats 4, 48 beats 35).
+// pt is sorted, so that run ends where the segment ends: a binary search for the end of j's
+// child run decides it.
+__global__ void k_lock_winner(const uint32_t *__restrict__ pt, uint64_t p, uint32_t lvl, uint32_t *__restrict__ win) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < p;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t sh = lvl ? lvl - 1 : 0;
+    const uint32_t c = pt[j] >> sh;
+    uint32_t w = 0;
+    if (j == 0 || (pt[j - 1] >> sh) != c) {            // first contender of its child run
+      if (lvl == 0) {
+        w = 1;
+      } else {
+        uint64_t lo = j + 1, hi = p;                   // first index past the child run
+        while (lo < hi) {
+          const uint64_t mid = (lo + hi) >> 1;
+          if ((pt[mid] >> sh) == c) lo = mid + 1;
+          else hi = mid;
+        }
+        w = (lo == p || (pt[lo] >> lvl) != (pt[j] >> lvl)) ? 1u : 0u;
+      }
+    }
+    win[j] = w;
+  }
+}
+
+// split at one level by the winner flags (hf) and their exclusive scan (widx): the winner of
+// every segment keeps going (winner list), the others abort to the next round (loser list,
+// appended at `na`)
 __global__ void k_lock_split(const uint64_t *__restrict__ pk, const uint32_t *__restrict__ pv,
                              const uint32_t *__restrict__ pt, const uint32_t *__restrict__ hf,
                              const uint32_t *__restrict__ widx, uint64_t p, uint64_t *__restrict__ wk,
@@ -1582,9 +1612,8 @@ __global__ void k_upd_summary(const uint32_t *__restrict__ pos, const uint32_t *
 }
 
 // GPMA concurrent insertion (Alg. 1): rounds of level-synchronous climbs with one
-// lock per segment.  Lock arbitration is deterministic -- the first (smallest-key) insertion
-// that reaches a segment wins it, the others abort to the next round -- so the layout is
-// reproducible (the oracle follows the same rule).  Winners test count + 1 <= max_i and are
+// lock per segment.  Lock arbitration is deterministic (R28, k_lock_winner) -- the others
+// abort to the next round -- so the layout is reproducible (the oracle follows the same rule).  Winners test count + 1 <= max_i and are
 // merged by the generic level step; a winner that reaches the root doubles it (l.20).
 static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
   gpma_status st;
@@ -1602,7 +1631,7 @@ static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
     uint64_t na = 0, nw = p, dirty_base = 0;
     for (uint32_t lvl = 0; lvl <= g->h && nw > 0; ++lvl) {   // the root is tested too (R6)
       Lvl a = make_lvl(g, cur, nw, lvl, GPMA_INSERT);
-      GP_LAUNCH(g, k_lvl_flags, grid_for(nw), TB, 0, s, a);
+      GP_LAUNCH(g, k_lock_winner, grid_for(nw), TB, 0, s, a.pt, nw, lvl, a.hf);
       scan_u32(g, a.hf, a.widx, nw, s);
       GP_LAUNCH(g, k_lock_split, grid_for(nw), TB, 0, s, a.pk, a.pv, a.pt, a.hf, a.widx, nw,
                 (uint64_t *)g->b_pk[cur ^ 1].p, (uint32_t *)g->b_pv[cur ^ 1].p, (uint32_t *)g->b_pt[cur ^ 1].p, ak,

@@ -9,7 +9,7 @@ import torch
 import oracle as O
 from gpma_gen import bfs_root, config_stream
 from gpma_gen.streams import StreamConfig
-from tests.gpu_helpers import DEV
+from tests.gpu_helpers import DEV, assert_pr_close
 
 pytestmark = pytest.mark.gpu
 
@@ -59,7 +59,8 @@ def test_concurrent_analytics_match_oracle():
             assert np.array_equal(lv.cpu().numpy(), ob), (step, rep)
             assert np.array_equal(lab.cpu().numpy().view(np.uint32), o.cc()), (step, rep)
             xo, _ = o.pagerank(tol=0.0, max_iter=5)
-            assert r[0] == 5 and np.abs(x.cpu().numpy() - xo).max() <= 1e-6, (step, rep)
+            assert r[0] == 5, (step, rep)
+            assert_pr_close(x.cpu().numpy(), xo, what=f"{step} {rep}")
             orp, ocol, oval = o.export_csr()
             assert r[3] == len(ocol)
             assert np.array_equal(rp.cpu().numpy().view(np.uint64), orp)

@@ -33,7 +33,7 @@ def _owned(keys, vals, V, P, r):
 def _run(rank, world, port, mode, seed, fails):
     import torch.distributed as dist
     from paper_journals_pvldb_shalht17_b200.dist import CudaShard, DistGpma, batch_slice, row_range
-    from tests.gpu_helpers import DEV, assert_same_layout
+    from tests.gpu_helpers import DEV, assert_pr_close, assert_same_layout
     try:
         if world > 1:
             os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
@@ -67,7 +67,8 @@ def _run(rank, world, port, mode, seed, fails):
             xt = None if x is None else torch.from_numpy(x.copy()).to(DEV)
             xg, it = dg.pagerank(xt, warm=x is not None, tol=0.0, max_iter=6)
             xo, _ = ref.pagerank(x=x, tol=0.0, max_iter=6)
-            assert it == 6 and np.abs(xg.cpu().numpy() - xo).max() <= 1e-6, "PR"
+            assert it == 6
+            assert_pr_close(xg.cpu().numpy(), xo, what="dist PR")
             x = xo
         if world > 1:
             dist.destroy_process_group()

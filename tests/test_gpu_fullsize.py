@@ -14,7 +14,8 @@ import torch
 import oracle as O
 from gpma_gen import CONFIGS, bfs_root, config_stream
 from gpma_gen.streams import StreamConfig, edge_values, make_stream
-from tests.gpu_helpers import (DEV, assert_same_csr, assert_same_layout, gpu_bfs, gpu_cc, gpu_pr)
+from tests.gpu_helpers import (DEV, assert_pr_close, assert_same_csr, assert_same_layout, gpu_bfs, gpu_cc,
+                               gpu_pr)
 
 pytestmark = [pytest.mark.gpu, pytest.mark.slow]
 
@@ -47,7 +48,9 @@ def test_config2_full_size():
     assert np.array_equal(gpu_cc(g), o.cc())
     xg, _ = gpu_pr(g, tol=0.0, max_iter=3)
     xo, _ = o.pagerank(tol=0.0, max_iter=3)
-    assert np.abs(xg - xo).max() <= 1e-6
+    assert_pr_close(xg, xo, what="config2 fp64")
+    x32, _ = gpu_pr(g, tol=0.0, max_iter=3, dtype=torch.float32)
+    assert_pr_close(x32, xo, fp64=False, what="config2 fp32")
 
 
 def test_config1_pokec_shaped_batch_sizes():

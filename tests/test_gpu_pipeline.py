@@ -6,7 +6,7 @@ import torch
 
 import oracle as O
 from gpma_gen import bfs_root, config_stream
-from tests.gpu_helpers import DEV
+from tests.gpu_helpers import DEV, assert_pr_close
 
 pytestmark = pytest.mark.gpu
 
@@ -40,6 +40,6 @@ def test_pipeline_matches_oracle(concurrent):
         assert np.array_equal(col.numpy().view(np.uint32), ocol)
         assert np.array_equal(cv.numpy().view(np.uint32), oval)
         xo, _ = o.pagerank(x=xo, tol=0.0, max_iter=100)
-        assert np.abs(x.numpy() - xo).max() <= 1e-6
+        assert_pr_close(x.numpy(), xo, what=f"slide {s}")
     pipe.drain()
     pipe.close()

@@ -20,6 +20,18 @@ def test_example2_round1_row(golden):
     assert _occ(o.dump()[0]) == g["round1_row"]
 
 
+def test_example2_full_batch_round1(golden):
+    """The FULL batch {1,4,9,35,48}, stopped after round 1: the Fig. 4 Round1 row -- 1 beats
+    4 for leaf 0 and 48 beats 35 for segment [24,31]; R28 reproduces both choices."""
+    g = golden("ex2_gpma_lock.json")
+    o = O.Oracle.raw(64, 32, 4, fig3_layout(), algorithm=1)
+    o.set_max_rounds(1)
+    o.insert(g["batch"], [0] * 5)
+    assert o.rounds == 1
+    assert _occ(o.dump()[0]) == g["round1_row"]
+    assert sorted(set(g["batch"]) - set(g["round1_row"])) == g["round1_losers"]
+
+
 def test_example2_full_batch_two_rounds(golden):
     """The full batch needs a second round for the aborted insertions (4 and one of 35/48)."""
     g = golden("ex2_gpma_lock.json")
