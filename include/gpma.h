@@ -82,6 +82,16 @@ typedef struct {
                                  (sources) [row_begin, row_end) only -- guards, row
                                  offsets and out-degrees for those rows; destinations
                                  range over [0, num_vertices).  0,0 = all rows.       */
+  /* Device memory of the store and of every scratch buffer (SURVEY §8(b) "Ownership"):
+   * alloc(bytes, stream, ctx) returns device memory usable in stream order on `stream`
+   * (NULL = out of memory -> GPMA_ERR_OOM); free(ptr, stream, ctx) releases it in stream
+   * order.  Both NULL (default) = a stream-ordered pool owned by the library (one per
+   * device, trimmed when the device's last handle is destroyed).  Set both or neither; the
+   * hooks must stay valid until gpma_destroy returns.  Added in the second version of this
+   * struct: callers compiled against the first (smaller struct_size) get the default.    */
+  void *(*alloc)(size_t bytes, gpma_stream_t stream, void *ctx);
+  void (*free)(void *ptr, gpma_stream_t stream, void *ctx);
+  void *alloc_ctx;
 } gpma_config;
 
 typedef struct {

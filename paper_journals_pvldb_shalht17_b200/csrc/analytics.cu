@@ -343,19 +343,19 @@ gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
 static gpma_status bfs_expand_level(gpma *g, Scratch &X, int32_t *levels, int32_t depth, const uint32_t *bm,
                                     uint32_t F, uint32_t *bm_next, uint32_t *fnext, cudaStream_t s) {
   const uint64_t V = g->V, nl = g->cap / g->L;
-  GP_CHECK(g, ensure(X.b[0], (V + 1) * 4, s));
-  GP_CHECK(g, ensure(X.misc, (nl + 2) * 4, s));
+  GP_CHECK(g, ensure(g, X.b[0], (V + 1) * 4, s));
+  GP_CHECK(g, ensure(g, X.misc, (nl + 2) * 4, s));
   uint32_t *list = (uint32_t *)X.b[0].p;
   uint32_t *alist = (uint32_t *)X.misc.p;
   uint32_t *cnt_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum2);   // list / active-leaf count
   const uint32_t *tmask = tmask_of(g);
   GP_CHECK(g, fill_zero(g, cnt_d, 4, s));
   if (F <= bfs_sparse_f()) {
-    GP_CHECK(g, ensure(X.b[2], ((uint64_t)bfs_sparse_f() + 2) * 8, s));   // fixed size: no regrowth per level
+    GP_CHECK(g, ensure(g, X.b[2], ((uint64_t)bfs_sparse_f() + 2) * 8, s));   // fixed size: no regrowth per level
     uint64_t *off = (uint64_t *)X.b[2].p;
     GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, cnt_d);
     GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, g->rb, g->nr, off);
-    scan_u64(g, off, off, F, s);
+    GP_CHECK(g, scan_u64(g, off, off, F, s));
     GP_LAUNCH(g, k_bfs_expand, grid_cap(), TA, 0, s, list, F, off, g->row_offset, g->key, tmask, g->L,
               levels, depth, g->rb, bm_next, fnext);
   } else {
@@ -406,7 +406,7 @@ gpma_status bfs_level(gpma *g, int32_t *levels, int32_t depth, uint32_t *frontie
   Scratch &X = g->an[AN_BFS];
   ScanScope scan_scope_(X.scan);
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(X.b[3], (V / 32 + 2) * 4, s));
+  GP_CHECK(g, ensure(g, X.b[3], (V / 32 + 2) * 4, s));
   uint32_t *bm = (uint32_t *)X.b[3].p;
   uint32_t *F_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum);
   GP_CHECK(g, fill_zero(g, F_d, 4, s));
@@ -425,8 +425,8 @@ gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
   Scratch &X = g->an[AN_BFS];
   ScanScope scan_scope_(X.scan);
   const uint64_t V = g->V, words = (V + 31) / 32 + 1;
-  GP_CHECK(g, ensure(X.b[3], words * 4, s));
-  GP_CHECK(g, ensure(X.b[1], words * 4, s));
+  GP_CHECK(g, ensure(g, X.b[3], words * 4, s));
+  GP_CHECK(g, ensure(g, X.b[1], words * 4, s));
   uint32_t *bm[2] = {(uint32_t *)X.b[3].p, (uint32_t *)X.b[1].p};
   uint32_t *F_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum);
   GP_CHECK(g, fill_zero(g, bm[0], words * 4, s));
@@ -708,7 +708,7 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
   Scratch &X = g->an[AN_CC];
   ScanScope scan_scope_(X.scan);
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(X.b[1], (V + 1) * 4, s));
+  GP_CHECK(g, ensure(g, X.b[1], (V + 1) * 4, s));
   uint32_t *prev = (uint32_t *)X.b[1].p;
   const uint32_t *tmask = tmask_of(g);
   if (init) GP_LAUNCH(g, k_cc_init, grid_for(V), TA, 0, s, labels, g->V);
@@ -731,7 +731,7 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
 gpma_status cc(gpma *g, uint32_t *labels, cudaStream_t s) {
   Scratch &X = g->an[AN_CC];
   ScanScope scan_scope_(X.scan);
-  GP_CHECK(g, ensure(X.b[0], ((uint64_t)g->V + 1) * 4, s));
+  GP_CHECK(g, ensure(g, X.b[0], ((uint64_t)g->V + 1) * 4, s));
   uint32_t *p = (uint32_t *)X.b[0].p;
   const uint32_t *tmask = tmask_of(g);
   GP_LAUNCH(g, k_cc_init, grid_for(g->V), TA, 0, s, p, g->V);
@@ -960,9 +960,9 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   ScanScope scan_scope_(X.scan);
   using A = typename PrAcc<T>::A;
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(X.b[1], (V + 1) * sizeof(A), s));
-  GP_CHECK(g, ensure(X.b[2], (V + 1) * sizeof(A), s));
-  GP_CHECK(g, ensure(X.b[3], 4 * sizeof(double) + sizeof(PrLoop), s));
+  GP_CHECK(g, ensure(g, X.b[1], (V + 1) * sizeof(A), s));
+  GP_CHECK(g, ensure(g, X.b[2], (V + 1) * sizeof(A), s));
+  GP_CHECK(g, ensure(g, X.b[3], 4 * sizeof(double) + sizeof(PrLoop), s));
   const uint32_t *deg = g->deg;
   A *contrib = (A *)X.b[1].p, *y = (A *)X.b[2].p;
   double *acc = (double *)X.b[3].p;   // [0],[1] dangling ping-pong, [2] error, then the loop state
@@ -1046,7 +1046,7 @@ __global__ void k_prd_update(double *__restrict__ x, unsigned long long *__restr
 gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s) {
   Scratch &X = g->an[AN_PR];
   ScanScope scan_scope_(X.scan);
-  GP_CHECK(g, ensure(X.b[1], ((uint64_t)g->nr + 1) * 8, s));
+  GP_CHECK(g, ensure(g, X.b[1], ((uint64_t)g->nr + 1) * 8, s));
   unsigned long long *contrib = (unsigned long long *)X.b[1].p;
   unsigned long long *yy = (unsigned long long *)y;
   if (init) GP_LAUNCH(g, k_prd_init, grid_for(g->V), TA, 0, s, x, g->V);
@@ -1254,10 +1254,10 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
   Scratch &X = g->an[AN_EXPORT];
   ScanScope scan_scope_(X.scan);
   const uint64_t nl = g->cap / g->L;
-  GP_CHECK(g, ensure(X.lpre, (nl + 1) * 8, s));
+  GP_CHECK(g, ensure(g, X.lpre, (nl + 1) * 8, s));
   uint64_t *lc = (uint64_t *)X.lpre.p;
   GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gcnt_of(g), nl, lc);
-  scan_u64(g, lc, lc, nl, s);
+  GP_CHECK(g, scan_u64(g, lc, lc, nl, s));
   GP_CHECK(g, readback(g, &X.ctrl_h->sum, lc + nl, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   uint64_t nnz = X.ctrl_h->sum;

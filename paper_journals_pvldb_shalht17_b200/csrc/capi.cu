@@ -34,11 +34,11 @@ struct Out {
   DevBuf buf;
   cudaStream_t s;
   Out(gpma *g_, void *u, size_t b, cudaStream_t s_) : g(g_), user(u), bytes(b), host(is_host_ptr(u)), s(s_) {}
-  ~Out() { gp::release(buf, s); }
+  ~Out() { gp::release(g, buf, s); }
   cudaError_t dev(void **p, bool copy_in) {
     if (!user) { *p = nullptr; return cudaSuccess; }
     if (!host) { *p = user; return cudaSuccess; }
-    cudaError_t e = gp::ensure(buf, bytes, s);
+    cudaError_t e = gp::ensure(g, buf, bytes, s);
     if (e) return e;
     if (copy_in) {
       e = cudaMemcpyAsync(buf.p, user, bytes, cudaMemcpyHostToDevice, s);
@@ -102,6 +102,11 @@ gpma_status apply_config(gpma *g, const gpma_config *cfg, uint32_t *leaf, uint64
     g->rb = 0;
     g->nr = g->V;
   }
+  if ((c.alloc == nullptr) != (c.free == nullptr)) return GPMA_ERR_INVALID_ARG;
+  g->alloc_fn = c.alloc;
+  g->free_fn = c.free;
+  g->alloc_ctx = c.alloc_ctx;
+  gp::pool_attach(g);
   *leaf = c.leaf_slots;
   *cap = c.initial_capacity;
   return GPMA_OK;
@@ -109,25 +114,7 @@ gpma_status apply_config(gpma *g, const gpma_config *cfg, uint32_t *leaf, uint64
 
 void free_handle(gpma *g);
 
-// Keep freed stream-ordered blocks in the device's default pool across synchronisations (the
-// default release threshold 0 returns them to the OS at every sync, so each regrowth of a
-// scratch buffer would map memory again).
-static void keep_pool_memory() {
-  static const bool done = [] {
-    int d = 0;
-    cudaMemPool_t pool;
-    if (cudaGetDevice(&d) == cudaSuccess && cudaDeviceGetDefaultMemPool(&pool, d) == cudaSuccess) {
-      uint64_t thr = ~0ull;
-      cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr);
-    }
-    cudaGetLastError();
-    return true;
-  }();
-  (void)done;
-}
-
 gpma *new_handle(uint32_t V) {
-  keep_pool_memory();
   gpma *g = new (std::nothrow) gpma();
   if (!g) return nullptr;
   g->V = V;
@@ -153,6 +140,10 @@ gpma *new_handle(uint32_t V) {
 
 void free_handle(gpma *g) {
   if (!g) return;
+  // analytics may still run on other streams (include/gpma.h "Concurrency"): let all of the
+  // device's work finish before the store and the scratch go back to the allocator
+  cudaDeviceSynchronize();
+  cudaGetLastError();
   cudaStream_t s = g->st;
   DevBuf *bufs[] = {&g->b_sk[0], &g->b_sk[1], &g->b_sv[0], &g->b_sv[1], &g->b_keep, &g->b_pos, &g->b_tgt,
                     &g->b_pk[0], &g->b_pk[1], &g->b_pv[0], &g->b_pv[1], &g->b_pt[0], &g->b_pt[1],
@@ -160,18 +151,19 @@ void free_handle(gpma *g) {
                     &g->b_woff, &g->b_keep2, &g->b_kpos, &g->b_lpre, &g->b_wk, &g->b_wv, &g->b_dirty,
                     &g->b_scan, &g->b_hist, &g->b_stage[0], &g->b_stage[1], &g->b_stage[2],
                     &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3};
-  for (DevBuf *b : bufs) gp::release(*b, s);
+  for (DevBuf *b : bufs) gp::release(g, *b, s);
   for (gp::Scratch &x : g->an) {
     DevBuf *xb[] = {&x.b[0], &x.b[1], &x.b[2], &x.b[3], &x.misc, &x.lpre, &x.scan, &x.stage[0], &x.stage[1]};
-    for (DevBuf *b : xb) gp::release(*b, s);
+    for (DevBuf *b : xb) gp::release(g, *b, s);
   }
-  if (g->key) cudaFreeAsync(g->key, s);
-  if (g->val) cudaFreeAsync(g->val, s);
-  if (g->cnt) cudaFreeAsync(g->cnt, s);
-  if (g->head) cudaFreeAsync(g->head, s);
-  if (g->row_offset) cudaFreeAsync(g->row_offset, s);
-  if (g->deg) cudaFreeAsync(g->deg, s);
+  gp::dev_free(g, g->key, s);
+  gp::dev_free(g, g->val, s);
+  gp::dev_free(g, g->cnt, s);
+  gp::dev_free(g, g->head, s);
+  gp::dev_free(g, g->row_offset, s);
+  gp::dev_free(g, g->deg, s);
   cudaStreamSynchronize(s);
+  gp::pool_detach(g);
   for (gp::UpdGraph &u : g->ugraph)
     if (u.exec) cudaGraphExecDestroy(u.exec);
   for (cudaEvent_t e : g->ev_pool) cudaEventDestroy(e);
@@ -254,10 +246,10 @@ gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t l
     g->h = gp::ilog2(capacity / leaf_slots);
     gp::level_bounds(g->L, g->h, g->rho0, g->rhoh, g->tau0, g->tauh, g->tmin, g->tmax);
     uint64_t nl = capacity / leaf_slots;
-    if (cudaMallocAsync((void **)&g->key, capacity * 8, s) || cudaMallocAsync((void **)&g->val, capacity * 4, s) ||
-        cudaMallocAsync((void **)&g->cnt, nl * 12, s) || cudaMallocAsync((void **)&g->head, nl * 8, s) ||
-        cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s) ||
-        cudaMallocAsync((void **)&g->deg, (uint64_t)g->nr * 4 + 4, s)) {
+    if (gp::dev_alloc(g, (void **)&g->key, capacity * 8, s) || gp::dev_alloc(g, (void **)&g->val, capacity * 4, s) ||
+        gp::dev_alloc(g, (void **)&g->cnt, nl * 12, s) || gp::dev_alloc(g, (void **)&g->head, nl * 8, s) ||
+        gp::dev_alloc(g, (void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s) ||
+        gp::dev_alloc(g, (void **)&g->deg, (uint64_t)g->nr * 4 + 4, s)) {
       cudaGetLastError();
       st = GPMA_ERR_OOM;
     }

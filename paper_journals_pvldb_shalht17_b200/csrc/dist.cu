@@ -21,8 +21,8 @@ gpma_status route(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t 
     for (uint32_t r = 0; r < nranks; ++r) counts_host[r] = 0;
     return GPMA_OK;
   }
-  GP_CHECK(g, ensure(g->b_stage[2], n * 8, s));
-  GP_CHECK(g, ensure(g->b_stage[3], n * 4 + 8 * (nranks + 1), s));
+  GP_CHECK(g, ensure(g, g->b_stage[2], n * 8, s));
+  GP_CHECK(g, ensure(g, g->b_stage[3], ((n * 4 + 7) & ~7ull) + 8 * (nranks + 1), s));   // vals, then starts (8-B aligned)
   uint64_t *k0 = (uint64_t *)g->b_stage[2].p;
   uint32_t *v0 = (uint32_t *)g->b_stage[3].p;
   uint64_t *starts = (uint64_t *)((char *)g->b_stage[3].p + ((n * 4 + 7) & ~7ull));

@@ -123,6 +123,13 @@ struct gpma {
   gp::Ctrl *ctrl_h = nullptr;     // pinned mirror
   gp::Scratch an[gp::AN_N];       // analytics (read-only on the store)
 
+  // device memory (gpma_config.alloc / free / alloc_ctx; NULL = the library's pool)
+  void *(*alloc_fn)(size_t, gpma_stream_t, void *) = nullptr;
+  void (*free_fn)(void *, gpma_stream_t, void *) = nullptr;
+  void *alloc_ctx = nullptr;
+  int device = 0;
+  bool pool_attached = false;
+
   // state
   bool poisoned = false;
   std::string err;
@@ -185,17 +192,23 @@ inline unsigned grid_for(uint64_t n, int block = 256, int max_blocks = 0) {
   return (unsigned)b;
 }
 
+// device memory of the library: the caller's hooks (gpma_config.alloc/free) or the
+// library-owned stream-ordered pool of the device
+cudaError_t dev_alloc(gpma *g, void **p, size_t bytes, cudaStream_t s);
+void dev_free(gpma *g, void *p, cudaStream_t s);
+void pool_attach(gpma *g);     // at create: pick the device's pool (counted per device)
+void pool_detach(gpma *g);     // at destroy: the last handle of a device trims its pool
 // allocate (stream-ordered) at least `bytes`, keeping the old block when large enough
-cudaError_t ensure(DevBuf &b, size_t bytes, cudaStream_t s);
-void release(DevBuf &b, cudaStream_t s);
+cudaError_t ensure(gpma *g, DevBuf &b, size_t bytes, cudaStream_t s);
+void release(gpma *g, DevBuf &b, cudaStream_t s);
 
 // exclusive scan: out[0..n) = prefix sums of in[0..n), out[n] = total.  in == out allowed.
-void scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s);
-void scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s);
-// stable LSD radix sort of (key, val) pairs on the given 8-bit digit shifts; returns
-// the index (0/1) of the buffer pair holding the result.
-int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1, uint64_t n,
-                     const int *shifts, int nshift, cudaStream_t s);
+[[nodiscard]] cudaError_t scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s);
+[[nodiscard]] cudaError_t scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s);
+// stable onesweep LSD radix sort of (key, val) pairs (vals may be null: keys only) on the
+// given 8-bit digit shifts; *which = the index (0/1) of the buffer pair holding the result.
+[[nodiscard]] cudaError_t radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1,
+                                           uint64_t n, const int *shifts, int nshift, cudaStream_t s, int *which);
 gpma_status radix_partition_owner(gpma *g, const uint64_t *k0, const uint32_t *v0, uint64_t *k1, uint32_t *v1,
                                   uint64_t n, uint32_t div, uint32_t nranks, uint64_t *starts_dev,
                                   cudaStream_t s);

@@ -13,24 +13,105 @@
 namespace gp {
 
 // ------------------------------------------------------------------ memory
-cudaError_t ensure(DevBuf &b, size_t bytes, cudaStream_t s) {
-  if (bytes == 0) bytes = 16;
-  if (b.bytes >= bytes) return cudaSuccess;
-  const size_t want = std::max(bytes, b.bytes + b.bytes / 2);  // grow x1.5 at least
-  if (b.p) cudaFreeAsync(b.p, s);
-  b.p = nullptr;
-  b.bytes = 0;
-  cudaError_t e = cudaMallocAsync(&b.p, want, s);
-  if (e != cudaSuccess) {
-    b.p = nullptr;
-    return e;
+// Every device allocation of the library goes through dev_alloc / dev_free: the caller's
+// hooks (gpma_config.alloc / free / alloc_ctx, e.g. PyTorch's caching allocator) when set,
+// else a stream-ordered allocation from a library-owned memory pool of the device.  The
+// pool keeps freed blocks mapped while any handle lives on the device (each regrowth of a
+// scratch buffer would otherwise map memory again) and is trimmed when the last handle of
+// the device is destroyed; the device's default pool (shared with every other
+// cudaMallocAsync user of the process) is left alone.
+namespace {
+std::mutex g_pool_mu;
+struct DevPool {
+  cudaMemPool_t pool = nullptr;
+  int handles = 0;
+};
+DevPool g_pools[64];
+}  // namespace
+
+static cudaMemPool_t lib_pool(int dev) {
+  std::lock_guard<std::mutex> lk(g_pool_mu);
+  DevPool &P = g_pools[dev & 63];
+  if (!P.pool) {
+    cudaMemPoolProps props{};
+    props.allocType = cudaMemAllocationTypePinned;
+    props.handleTypes = cudaMemHandleTypeNone;
+    props.location.type = cudaMemLocationTypeDevice;
+    props.location.id = dev;
+    if (cudaMemPoolCreate(&P.pool, &props) != cudaSuccess) {
+      cudaGetLastError();
+      P.pool = nullptr;
+      return nullptr;
+    }
+    uint64_t thr = ~0ull;
+    cudaMemPoolSetAttribute(P.pool, cudaMemPoolAttrReleaseThreshold, &thr);
   }
-  b.bytes = want;
-  return cudaSuccess;
+  return P.pool;
 }
 
-void release(DevBuf &b, cudaStream_t s) {
-  if (b.p) cudaFreeAsync(b.p, s);
+void pool_attach(gpma *g) {
+  if (g->alloc_fn) return;
+  cudaGetDevice(&g->device);
+  lib_pool(g->device);
+  std::lock_guard<std::mutex> lk(g_pool_mu);
+  g_pools[g->device & 63].handles++;
+  g->pool_attached = true;
+}
+
+void pool_detach(gpma *g) {
+  if (!g->pool_attached) return;
+  std::lock_guard<std::mutex> lk(g_pool_mu);
+  DevPool &P = g_pools[g->device & 63];
+  if (--P.handles == 0 && P.pool) cudaMemPoolTrimTo(P.pool, 0);   // every block is free by now
+  g->pool_attached = false;
+}
+
+cudaError_t dev_alloc(gpma *g, void **p, size_t bytes, cudaStream_t s) {
+  *p = nullptr;
+  if (g->alloc_fn) {
+    *p = g->alloc_fn(bytes, (gpma_stream_t)s, g->alloc_ctx);
+    return *p ? cudaSuccess : cudaErrorMemoryAllocation;
+  }
+  cudaMemPool_t pool = lib_pool(g->device);
+  cudaError_t e = pool ? cudaMallocFromPoolAsync(p, bytes, pool, s) : cudaMallocAsync(p, bytes, s);
+  if (e != cudaSuccess) {
+    cudaGetLastError();
+    *p = nullptr;
+  }
+  return e;
+}
+
+void dev_free(gpma *g, void *p, cudaStream_t s) {
+  if (!p) return;
+  if (g->alloc_fn) {
+    if (g->free_fn) g->free_fn(p, (gpma_stream_t)s, g->alloc_ctx);
+    return;
+  }
+  cudaFreeAsync(p, s);
+}
+
+// At least `bytes` in b (grown x1.5 to amortise regrowth; on failure retried at exactly
+// `bytes`).  On failure b is empty and the error is returned: every caller checks it.
+cudaError_t ensure(gpma *g, DevBuf &b, size_t bytes, cudaStream_t s) {
+  if (bytes == 0) bytes = 16;
+  if (b.bytes >= bytes) return cudaSuccess;
+  const size_t want = std::max(bytes, b.bytes + b.bytes / 2);
+  dev_free(g, b.p, s);
+  b.p = nullptr;
+  b.bytes = 0;
+  cudaError_t e = dev_alloc(g, &b.p, want, s);
+  if (e != cudaSuccess && want > bytes) {
+    e = dev_alloc(g, &b.p, bytes, s);
+    if (e == cudaSuccess) b.bytes = bytes;
+  } else if (e == cudaSuccess) {
+    b.bytes = want;
+  }
+  if (e != cudaSuccess) b.p = nullptr;
+  return e;
+}
+
+void release(gpma *g, DevBuf &b, cudaStream_t s) {
+  dev_free(g, b.p, s);
   b.p = nullptr;
   b.bytes = 0;
 }
@@ -317,25 +398,27 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
 }
 
 template <typename T>
-static void scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) {
+static cudaError_t scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) {
   const uint64_t nt = (n + SC_TILE - 1) / SC_TILE > 0 ? (n + SC_TILE - 1) / SC_TILE : 1;
   if (nt == 1) {                       // one tile: no look-back, no status reset
     GP_LAUNCH(g, k_scan_lookback<T>, 1, SC_THREADS, 0, s, in, out, n, (unsigned long long *)nullptr);
-    return;
+    return cudaGetLastError();
   }
   DevBuf &sb = tl_scan ? *tl_scan : g->b_scan;
-  ensure(sb, (nt + 1) * sizeof(unsigned long long), s);
+  cudaError_t e = ensure(g, sb, (nt + 1) * sizeof(unsigned long long), s);
+  if (e != cudaSuccess) return e;
   unsigned long long *status = (unsigned long long *)sb.p;
-  fill_zero(g, status, (nt + 1) * sizeof(unsigned long long), s);
+  if ((e = fill_zero(g, status, (nt + 1) * sizeof(unsigned long long), s)) != cudaSuccess) return e;
   GP_LAUNCH(g, k_scan_lookback<T>, (unsigned)nt, SC_THREADS, 0, s, in, out, n, status);
+  return cudaGetLastError();
 }
 
-void scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s) {
-  scan_impl<uint32_t>(g, in, out, n, s);
+cudaError_t scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s) {
+  return scan_impl<uint32_t>(g, in, out, n, s);
 }
 
-void scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s) {
-  scan_impl<uint64_t>(g, in, out, n, s);
+cudaError_t scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s) {
+  return scan_impl<uint64_t>(g, in, out, n, s);
 }
 
 // ------------------------------------------------------------------ radix sort
@@ -462,28 +545,238 @@ __global__ void __launch_bounds__(1024) k_small_sort(uint64_t *k0, uint32_t *v0,
   }
 }
 
-int radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1, uint64_t n,
-                     const int *shifts, int nshift, cudaStream_t s) {
-  if (n <= 1) return 0;
-  if (n <= (uint64_t)SS_MAX) {
-    GP_LAUNCH(g, k_small_sort, 1, 1024, 0, s, k0, v0, k1, v1, (uint32_t)n);
-    return 1;
+// ---- onesweep LSD radix sort (the sort of every update batch, Alg. 4 l.2)
+// One read of the keys builds the digit histograms of every pass (k_os_hist); then each pass is
+// ONE kernel (k_os_pass): a CTA takes the next 4096-key tile (tile ids from an atomic counter,
+// so every predecessor is already resident), ranks its keys stably per warp (__match_any_sync
+// peer groups, in input order), publishes its per-digit counts and walks back over the
+// predecessors' published (aggregate | inclusive) counts digit by digit (decoupled look-back),
+// reorders the tile by digit in shared memory and writes each digit's run contiguously.
+// 2 + passes launches per sort instead of 4 per pass (hist, zero, scan, scatter), and the
+// batch (12 B per key, <= 12 MiB at 2^20) stays L2-resident across the passes.
+// Status words: [flag:2 | count:62]; flag 0 = not ready, 1 = tile aggregate, 2 = inclusive prefix.
+// Two status regions alternate between passes: the histogram kernel zeroes both (ntiles x 256
+// words each), and pass p's tile t zeroes its slot of the region pass p-1 used, which pass p+1
+// uses next -- so every pass finds its region zero with no host-side state (graph-replay safe).
+constexpr int OS_T = 256, OS_I = 16, OS_TILE = OS_T * OS_I, OS_W = OS_T / 32;
+constexpr int OS_MAXPASS = 8;
+struct OsPasses {
+  int shift[OS_MAXPASS];
+  int n;
+};
+constexpr uint64_t OS_CNT_MASK = (1ull << 62) - 1;
+constexpr size_t OS_SMEM = (size_t)OS_TILE * 8 + (size_t)OS_TILE * 4 + (size_t)OS_W * 256 * 4 + 256 * 4 * 2 + 256 * 8;
+
+__global__ void __launch_bounds__(OS_T) k_os_hist(const uint64_t *__restrict__ keys, uint64_t n, OsPasses ps,
+                                                  uint32_t *__restrict__ ghist, uint4 *__restrict__ status,
+                                                  uint64_t status_words16) {
+  __shared__ uint32_t h[OS_MAXPASS][256];
+  for (int i = threadIdx.x; i < OS_MAXPASS * 256; i += OS_T) (&h[0][0])[i] = 0;
+  for (uint64_t i = blockIdx.x * (uint64_t)OS_T + threadIdx.x; i < status_words16; i += (uint64_t)gridDim.x * OS_T)
+    status[i] = make_uint4(0, 0, 0, 0);               // both status regions
+  __syncthreads();
+  const uint64_t stride = (uint64_t)gridDim.x * OS_T * 2;
+  for (uint64_t i = (blockIdx.x * (uint64_t)OS_T + threadIdx.x) * 2; i < n; i += stride) {
+    uint64_t k0, k1 = 0;
+    const bool two = i + 1 < n;
+    if (two) {
+      const ulonglong2 kk = __ldg(reinterpret_cast<const ulonglong2 *>(keys + i));
+      k0 = kk.x;
+      k1 = kk.y;
+    } else {
+      k0 = keys[i];
+    }
+    for (int p = 0; p < ps.n; ++p) {
+      atomicAdd(&h[p][(uint32_t)(k0 >> ps.shift[p]) & 255u], 1u);
+      if (two) atomicAdd(&h[p][(uint32_t)(k1 >> ps.shift[p]) & 255u], 1u);
+    }
   }
-  const uint32_t ntiles = (uint32_t)((n + RS_TILE - 1) / RS_TILE);
-  const uint64_t hn = (uint64_t)ntiles * 256;
-  ensure(g->b_hist, (hn + 1) * sizeof(uint32_t), s);
-  uint32_t *hist = (uint32_t *)g->b_hist.p;
+  __syncthreads();
+  for (int i = threadIdx.x; i < ps.n * 256; i += OS_T) {
+    const uint32_t c = (&h[0][0])[i];
+    if (c) atomicAdd(ghist + i, c);
+  }
+}
+
+template <bool HASV>
+__global__ void __launch_bounds__(OS_T, 2) k_os_pass(const uint64_t *__restrict__ kin, const uint32_t *__restrict__ vin,
+                                                     uint64_t *__restrict__ kout, uint32_t *__restrict__ vout,
+                                                     uint64_t n, int shift, const uint32_t *__restrict__ ghist,
+                                                     unsigned long long *status, unsigned long long *status_prev,
+                                                     uint32_t *tile_ctr) {
+  extern __shared__ __align__(16) unsigned char os_smem[];
+  uint64_t *sk = reinterpret_cast<uint64_t *>(os_smem);                           // [OS_TILE]
+  uint32_t *sv = reinterpret_cast<uint32_t *>(sk + OS_TILE);                      // [OS_TILE]
+  uint32_t *wc = sv + OS_TILE;                                                    // [OS_W][256]
+  uint32_t *ldoff = wc + OS_W * 256;                                              // [256]
+  uint32_t *sbase = ldoff + 256;                                                  // [256] (digit bases, then tile id)
+  uint64_t *gofs = reinterpret_cast<uint64_t *>(sbase + 256);                     // [256]
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5, t = threadIdx.x;
+  const uint32_t lt = (1u << lane) - 1u;
+  for (int i = t; i < OS_W * 256; i += OS_T) wc[i] = 0;
+  // exclusive scan of the pass's global digit histogram (digit t) -> bases of the digit runs
+  const uint32_t gh = ghist[t];
+  {
+    uint32_t x = gh;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+      if (lane >= o) x += y;
+    }
+    if (lane == 31) ldoff[w] = x;                    // warp totals (ldoff reused as scratch)
+    __syncthreads();
+    uint32_t pre = 0;
+    for (int k = 0; k < w; ++k) pre += ldoff[k];
+    sbase[t] = pre + x - gh;
+  }
+  if (t == 0) ldoff[OS_W] = atomicAdd(tile_ctr, 1u);   // the tile of this CTA
+  __syncthreads();
+  const uint64_t tile = ldoff[OS_W];
+  const uint64_t dbase = sbase[t];
+  if (status_prev) status_prev[tile * 256 + t] = 0ull;   // the region pass p+1 uses (pass p-1 is done)
+  __syncthreads();
+  const uint64_t t0 = tile * OS_TILE;
+  const uint64_t base = t0 + (uint64_t)w * (32 * OS_I);
+  uint64_t k[OS_I];
+  uint32_t v[OS_I], r[OS_I];
+#pragma unroll
+  for (int j = 0; j < OS_I; ++j) {
+    const uint64_t i = base + j * 32 + lane;
+    k[j] = i < n ? kin[i] : 0ull;
+    if (HASV) v[j] = i < n ? vin[i] : 0u;
+  }
+  // stable per-warp ranks in input order (j-major, lane-minor)
+#pragma unroll
+  for (int j = 0; j < OS_I; ++j) {
+    const uint64_t i = base + j * 32 + lane;
+    const bool ok = i < n;
+    const uint32_t d = ok ? (uint32_t)(k[j] >> shift) & 255u : 256u + lane;
+    const uint32_t peers = __match_any_sync(0xffffffffu, d);
+    const uint32_t cur = ok ? wc[w * 256 + d] : 0u;
+    __syncwarp();
+    const uint32_t rank = __popc(peers & lt);
+    if (ok && rank == 0) wc[w * 256 + d] = cur + __popc(peers);
+    __syncwarp();
+    r[j] = cur + rank;
+  }
+  __syncthreads();
+  // digit t: offsets of the warps inside the tile, tile count
+  uint32_t run = 0;
+#pragma unroll
+  for (int ww = 0; ww < OS_W; ++ww) {
+    const uint32_t c = wc[ww * 256 + t];
+    wc[ww * 256 + t] = run;
+    run += c;
+  }
+  // publish the tile's aggregate for digit t, then look back for the exclusive prefix
+  volatile unsigned long long *st = status;
+  {
+    const unsigned long long word = ((tile == 0 ? 2ull : 1ull) << 62) | (unsigned long long)run;
+    __threadfence();
+    st[tile * 256 + t] = word;
+  }
+  uint64_t excl = 0;
+  for (int64_t p = (int64_t)tile - 1; p >= 0; --p) {
+    unsigned long long x;
+    do {
+      x = st[(uint64_t)p * 256 + t];
+    } while ((x >> 62) == 0);
+    excl += x & OS_CNT_MASK;
+    if ((x >> 62) == 2) break;
+  }
+  if (tile) {
+    __threadfence();
+    st[tile * 256 + t] = (2ull << 62) | (unsigned long long)(excl + run);
+  }
+  // local digit offsets inside the tile (exclusive scan of the tile counts over digits)
+  {
+    uint32_t x = run;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+      if (lane >= o) x += y;
+    }
+    __syncthreads();                                 // (sbase is free again)
+    if (lane == 31) sbase[w] = x;
+    __syncthreads();
+    uint32_t pre = 0;
+    for (int kk = 0; kk < w; ++kk) pre += sbase[kk];
+    ldoff[t] = pre + x - run;
+    gofs[t] = dbase + excl;
+  }
+  __syncthreads();
+  // reorder the tile by digit in shared memory
+#pragma unroll
+  for (int j = 0; j < OS_I; ++j) {
+    const uint64_t i = base + j * 32 + lane;
+    if (i < n) {
+      const uint32_t d = (uint32_t)(k[j] >> shift) & 255u;
+      const uint32_t lp = ldoff[d] + wc[w * 256 + d] + r[j];
+      sk[lp] = k[j];
+      if (HASV) sv[lp] = v[j];
+    }
+  }
+  __syncthreads();
+  // write each digit's run contiguously
+  const uint32_t nt = (uint32_t)min((uint64_t)OS_TILE, n - t0);
+#pragma unroll 4
+  for (uint32_t i = t; i < nt; i += OS_T) {
+    const uint64_t kk = sk[i];
+    const uint32_t d = (uint32_t)(kk >> shift) & 255u;
+    const uint64_t pos = gofs[d] + (i - ldoff[d]);
+    kout[pos] = kk;
+    if (HASV) vout[pos] = sv[i];
+  }
+}
+
+// Sort (k0, v0)[0..n) by the given 8-bit digit shifts (stable); v0 == nullptr sorts keys only.
+// *which = the buffer pair (0: k0/v0, 1: k1/v1) holding the result.
+cudaError_t radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1, uint64_t n,
+                             const int *shifts, int nshift, cudaStream_t s, int *which) {
+  *which = 0;
+  if (n <= 1 || nshift == 0) return cudaSuccess;
+  if (n <= (uint64_t)SS_MAX && v0) {
+    GP_LAUNCH(g, k_small_sort, 1, 1024, 0, s, k0, v0, k1, v1, (uint32_t)n);
+    *which = 1;
+    return cudaGetLastError();
+  }
+  static const bool attr = [] {
+    cudaFuncSetAttribute(k_os_pass<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)OS_SMEM);
+    cudaFuncSetAttribute(k_os_pass<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)OS_SMEM);
+    return true;
+  }();
+  (void)attr;
+  const uint64_t ntiles = (n + OS_TILE - 1) / OS_TILE;
+  const size_t ctl = 64 + (size_t)OS_MAXPASS * 256 * 4;        // tile counters + histograms
+  const uint64_t region = ntiles * 256;                         // status words per region
+  cudaError_t e = ensure(g, g->b_hist, ctl + 2 * region * 8, s);
+  if (e != cudaSuccess) return e;
+  char *base = (char *)g->b_hist.p;
+  uint32_t *ctr = (uint32_t *)base;
+  uint32_t *ghist = (uint32_t *)(base + 64);
+  unsigned long long *status = (unsigned long long *)(base + ctl);
+  if ((e = fill_zero(g, base, ctl, s)) != cudaSuccess) return e;
+  OsPasses ps{};
+  ps.n = nshift;
+  for (int p = 0; p < nshift; ++p) ps.shift[p] = shifts[p];
+  GP_LAUNCH(g, k_os_hist, grid_for((n + 1) / 2, OS_T, num_sms() * 4), OS_T, 0, s, k0, n, ps, ghist,
+            (uint4 *)status, region * 2 * 8 / 16);
   uint64_t *ks[2] = {k0, k1};
   uint32_t *vs[2] = {v0, v1};
   int cur = 0;
   for (int p = 0; p < nshift; ++p) {
-    GP_LAUNCH(g, k_radix_hist, ntiles, RS_THREADS, 0, s, ks[cur], n, shifts[p], hist, ntiles, 0u);
-    scan_u32(g, hist, hist, hn, s);
-    GP_LAUNCH(g, k_radix_scatter, ntiles, RS_THREADS, 0, s, ks[cur], vs[cur], ks[cur ^ 1],
-              vs[cur ^ 1], n, shifts[p], hist, ntiles, 0u);
+    unsigned long long *sp = status + (uint64_t)(p & 1) * region;
+    unsigned long long *sq = p ? status + (uint64_t)((p - 1) & 1) * region : nullptr;
+    if (v0)
+      GP_LAUNCH(g, k_os_pass<true>, (unsigned)ntiles, OS_T, OS_SMEM, s, ks[cur], vs[cur], ks[cur ^ 1], vs[cur ^ 1], n,
+                shifts[p], ghist + p * 256, sp, sq, ctr + p);
+    else
+      GP_LAUNCH(g, k_os_pass<false>, (unsigned)ntiles, OS_T, OS_SMEM, s, ks[cur], (const uint32_t *)nullptr,
+                ks[cur ^ 1], (uint32_t *)nullptr, n, shifts[p], ghist + p * 256, sp, sq, ctr + p);
     cur ^= 1;
   }
-  return cur;
+  *which = cur;
+  return cudaGetLastError();
 }
 
 __global__ void k_owner_starts(const uint32_t *__restrict__ hscan, uint32_t ntiles, uint32_t nranks,
@@ -498,10 +791,10 @@ gpma_status radix_partition_owner(gpma *g, const uint64_t *k0, const uint32_t *v
                                   cudaStream_t s) {
   const uint32_t ntiles = (uint32_t)std::max<uint64_t>(1, (n + RS_TILE - 1) / RS_TILE);
   const uint64_t hn = (uint64_t)ntiles * 256;
-  GP_CHECK(g, ensure(g->b_hist, (hn + 1) * sizeof(uint32_t), s));
-  uint32_t *hist = (uint32_t *)g->b_hist.p;
+  GP_CHECK(g, ensure(g, g->b_misc3, (hn + 1) * sizeof(uint32_t), s));
+  uint32_t *hist = (uint32_t *)g->b_misc3.p;
   GP_LAUNCH(g, k_radix_hist, ntiles, RS_THREADS, 0, s, k0, n, 0, hist, ntiles, div);
-  scan_u32(g, hist, hist, hn, s);
+  GP_CHECK(g, scan_u32(g, hist, hist, hn, s));
   GP_LAUNCH(g, k_radix_scatter, ntiles, RS_THREADS, 0, s, k0, v0, k1, v1, n, 0, hist, ntiles, div);
   GP_LAUNCH(g, k_owner_starts, 1, 256, 0, s, hist, ntiles, nranks, n, starts_dev);
   GP_CHECK(g, cudaGetLastError());

@@ -155,7 +155,7 @@ gpma_status query_edges(gpma *g, const uint64_t *keys, uint64_t n, uint32_t *val
   Scratch &X = g->an[AN_QUERY];
   ScanScope scan_scope_(X.scan);
   if (!n) return GPMA_OK;
-  GP_CHECK(g, ensure(X.stage[0], n * 8, s));
+  GP_CHECK(g, ensure(g, X.stage[0], n * 8, s));
   uint64_t *q = (uint64_t *)X.stage[0].p;
   GP_CHECK(g, stage_in(g, q, keys, n * 8, s));
   GP_LAUNCH(g, k_query_edges, grid_for(n), TQ, 0, s, q, n, g->key, g->val, g->head, (uint32_t)(g->cap / g->L),
@@ -168,13 +168,13 @@ gpma_status query_neighbors(gpma *g, const uint32_t *verts, uint64_t n, uint64_t
                             uint32_t *val, uint64_t cap_nnz, uint64_t *nnz_out, cudaStream_t s) {
   Scratch &X = g->an[AN_QUERY];
   ScanScope scan_scope_(X.scan);
-  GP_CHECK(g, ensure(X.stage[1], (n + 1) * 4, s));
-  GP_CHECK(g, ensure(X.lpre, (n + 1) * 8, s));
+  GP_CHECK(g, ensure(g, X.stage[1], (n + 1) * 4, s));
+  GP_CHECK(g, ensure(g, X.lpre, (n + 1) * 8, s));
   uint32_t *vq = (uint32_t *)X.stage[1].p;
   uint64_t *rp = (uint64_t *)X.lpre.p;
   if (n) GP_CHECK(g, stage_in(g, vq, verts, n * 4, s));
   if (n) GP_LAUNCH(g, k_query_rowsizes, grid_for(n), TQ, 0, s, vq, n, g->deg, g->rb, g->nr, rp);
-  scan_u64(g, rp, rp, n, s);
+  GP_CHECK(g, scan_u64(g, rp, rp, n, s));
   GP_CHECK(g, readback(g, &X.ctrl_h->sum, rp + n, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   const uint64_t nnz = n ? X.ctrl_h->sum : 0;
@@ -197,10 +197,10 @@ gpma_status query_reachable(gpma *g, const uint32_t *src, const uint32_t *dst, u
   Scratch &X = g->an[AN_QUERY];
   ScanScope scan_scope_(X.scan);
   const uint64_t V = g->V;
-  GP_CHECK(g, ensure(X.b[0], V * 8, s));
-  GP_CHECK(g, ensure(X.b[1], V * 8, s));
-  GP_CHECK(g, ensure(X.b[2], V * 8, s));
-  GP_CHECK(g, ensure(X.stage[1], 2 * 64 * 4 + 16, s));
+  GP_CHECK(g, ensure(g, X.b[0], V * 8, s));
+  GP_CHECK(g, ensure(g, X.b[1], V * 8, s));
+  GP_CHECK(g, ensure(g, X.b[2], V * 8, s));
+  GP_CHECK(g, ensure(g, X.stage[1], 2 * 64 * 4 + 16, s));
   unsigned long long *seen = (unsigned long long *)X.b[0].p, *front = (unsigned long long *)X.b[1].p,
                      *next = (unsigned long long *)X.b[2].p;
   uint32_t *qs = (uint32_t *)X.stage[1].p, *qd = qs + 64;

@@ -1086,16 +1086,17 @@ static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v
                                uint64_t **hd, cudaStream_t s) {
   uint64_t nl = cap / g->L;
   *k = nullptr; *v = nullptr; *c = nullptr; *hd = nullptr;
-  cudaError_t e1 = cudaMallocAsync((void **)k, cap * 8, s);
-  cudaError_t e2 = cudaMallocAsync((void **)v, cap * 4, s);
-  cudaError_t e3 = cudaMallocAsync((void **)c, nl * 12, s);  // live counts, tombstone masks, guards
-  cudaError_t e4 = cudaMallocAsync((void **)hd, nl * 8, s);
+  cudaError_t e1 = dev_alloc(g, (void **)k, cap * 8, s);
+  cudaError_t e2 = dev_alloc(g, (void **)v, cap * 4, s);
+  cudaError_t e3 = dev_alloc(g, (void **)c, nl * 12, s);  // live counts, tombstone masks, guards
+  cudaError_t e4 = dev_alloc(g, (void **)hd, nl * 8, s);
   if (e1 || e2 || e3 || e4) {
     cudaGetLastError();
-    if (*k) cudaFreeAsync(*k, s);
-    if (*v) cudaFreeAsync(*v, s);
-    if (*c) cudaFreeAsync(*c, s);
-    if (*hd) cudaFreeAsync(*hd, s);
+    dev_free(g, *k, s);
+    dev_free(g, *v, s);
+    dev_free(g, *c, s);
+    dev_free(g, *hd, s);
+    *k = nullptr; *v = nullptr; *c = nullptr; *hd = nullptr;
     g->err = "out of device memory allocating the store";
     return GPMA_ERR_OOM;
   }
@@ -1130,10 +1131,10 @@ gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaSt
 // key; returns the number of unique keys in *m, result in b_sk[0]/b_sv[0].
 static gpma_status sort_unique(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
                                uint64_t *m, bool need_unique_compact, int *which, cudaStream_t s) {
-  GP_CHECK(g, ensure(g->b_sk[0], n * 8, s));
-  GP_CHECK(g, ensure(g->b_sk[1], n * 8, s));
-  GP_CHECK(g, ensure(g->b_sv[0], n * 4, s));
-  GP_CHECK(g, ensure(g->b_sv[1], n * 4, s));
+  GP_CHECK(g, ensure(g, g->b_sk[0], n * 8, s));
+  GP_CHECK(g, ensure(g, g->b_sk[1], n * 8, s));
+  GP_CHECK(g, ensure(g, g->b_sv[0], n * 4, s));
+  GP_CHECK(g, ensure(g, g->b_sv[1], n * 4, s));
   uint64_t *k0 = (uint64_t *)g->b_sk[0].p, *k1 = (uint64_t *)g->b_sk[1].p;
   uint32_t *v0 = (uint32_t *)g->b_sv[0].p, *v1 = (uint32_t *)g->b_sv[1].p;
   GP_CHECK(g, stage_in(g, k0, keys, n * 8, s));
@@ -1141,7 +1142,7 @@ static gpma_status sort_unique(gpma *g, const uint64_t *keys, const uint32_t *va
   else GP_CHECK(g, fill_zero(g, v0, n * 4, s));
   int sh[8];
   int ns = key_shifts(g->V, sh);
-  *which = radix_sort_pairs(g, k0, v0, k1, v1, n, sh, ns, s);
+  GP_CHECK(g, radix_sort_pairs(g, k0, v0, k1, v1, n, sh, ns, s, which));
   (void)need_unique_compact;
   *m = n;
   GP_CHECK(g, cudaGetLastError());
@@ -1168,8 +1169,8 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
   const uint32_t *ev = nullptr;
   if (n) {
     // stage + validate on device
-    GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
-    GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
+    GP_CHECK(g, ensure(g, g->b_stage[0], n * 8, s));
+    GP_CHECK(g, ensure(g, g->b_stage[1], n * 4, s));
     GP_CHECK(g, stage_in(g, g->b_stage[0].p, keys, n * 8, s));
     GP_CHECK(g, stage_in(g, g->b_stage[1].p, vals, n * 4, s));
     if ((st = validate(g, (uint64_t *)g->b_stage[0].p, (uint32_t *)g->b_stage[1].p, n, true, s)))
@@ -1181,11 +1182,11 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
       return st;
     uint64_t *sk = (uint64_t *)g->b_sk[which].p;
     uint32_t *sv = (uint32_t *)g->b_sv[which].p;
-    GP_CHECK(g, ensure(g->b_keep, (n + 1) * 4, s));
-    GP_CHECK(g, ensure(g->b_pos, (n + 1) * 4, s));
+    GP_CHECK(g, ensure(g, g->b_keep, (n + 1) * 4, s));
+    GP_CHECK(g, ensure(g, g->b_pos, (n + 1) * 4, s));
     uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p;
     GP_LAUNCH(g, k_unique_last, grid_for(n), TB, 0, s, sk, n, keep);
-    scan_u32(g, keep, pos, n, s);
+    GP_CHECK(g, scan_u32(g, keep, pos, n, s));
     uint32_t mh = 0;
     GP_CHECK(g, readback(g, &g->ctrl_h->sum, pos + n, 4, s));
     GP_CHECK(g, cudaStreamSynchronize(s));
@@ -1215,16 +1216,16 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
   }
   set_geometry(g, cap);
   if ((st = alloc_store(g, cap, &g->key, &g->val, &g->cnt, &g->head, s))) return st;
-  GP_CHECK(g, cudaMallocAsync((void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s));
+  GP_CHECK(g, dev_alloc(g, (void **)&g->row_offset, ((uint64_t)g->nr + 1) * 8, s));
   GP_CHECK(g, fill_zero(g, g->row_offset, ((uint64_t)g->nr + 1) * 8, s));
-  GP_CHECK(g, cudaMallocAsync((void **)&g->deg, (uint64_t)g->nr * 4 + 4, s));
+  GP_CHECK(g, dev_alloc(g, (void **)&g->deg, (uint64_t)g->nr * 4 + 4, s));
   if (E > g->tmax[g->h] && !cap_override) {
     g->err = "initial graph exceeds the root bound";
     return GPMA_ERR_INVALID_ARG;
   }
   // dense merged list (edges + guards) in the window scratch
-  GP_CHECK(g, ensure(g->b_wk, std::max<uint64_t>(E, 1) * 8, s));
-  GP_CHECK(g, ensure(g->b_wv, std::max<uint64_t>(E, 1) * 4, s));
+  GP_CHECK(g, ensure(g, g->b_wk, std::max<uint64_t>(E, 1) * 8, s));
+  GP_CHECK(g, ensure(g, g->b_wv, std::max<uint64_t>(E, 1) * 4, s));
   uint64_t *wk = (uint64_t *)g->b_wk.p;
   uint32_t *wv = (uint32_t *)g->b_wv.p;
   if (m) {
@@ -1233,7 +1234,7 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
     // recompute from the dense list: keep = 1, pos = j
     // (the dense list ek is sorted & unique; place directly)
     GP_LAUNCH(g, k_unique_last, grid_for(m), TB, 0, s, ek, m, keep);  // all ones (unique)
-    scan_u32(g, keep, pos, m, s);
+    GP_CHECK(g, scan_u32(g, keep, pos, m, s));
     GP_LAUNCH(g, k_place_edges, grid_for(m), TB, 0, s, ek, ev, pos, keep, m, wk, wv, g->rb);
   }
   GP_LAUNCH(g, k_place_guards, grid_for(g->nr), TB, 0, s, g->rb, g->nr, ek, m, wk, wv);
@@ -1266,7 +1267,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     GP_LAUNCH(g, k_lvl_front_small, 1, LS_T, 0, s, a, g->cnt);
   } else {
   GP_LAUNCH(g, k_lvl_flags, gp, TB, 0, s, a);
-  scan_u32(g, a.hf, a.widx, p, s);
+  GP_CHECK(g, scan_u32(g, a.hf, a.widx, p, s));
   GP_LAUNCH(g, k_lvl_first, gp, TB, 0, s, a);
   if (a.lvl <= 4) GP_LAUNCH(g, k_lvl_count<1>, grid_for(p), TB, 0, s, a, g->cnt);
   else if (a.lvl <= 11) GP_LAUNCH(g, k_lvl_count<32>, grid_for(p * 32), TB, 0, s, a, g->cnt);
@@ -1278,8 +1279,8 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
               chunk);
     GP_LAUNCH(g, k_lvl_accept, gp, TB, 0, s, a);
   }
-  scan_u32(g, a.acc, a.aidx, p, s);
-  scan_u64(g, a.nw, a.woff, p, s);
+  GP_CHECK(g, scan_u32(g, a.acc, a.aidx, p, s));
+  GP_CHECK(g, scan_u64(g, a.nw, a.woff, p, s));
   GP_LAUNCH(g, k_lvl_alist, gp, TB, 0, s, a);
   }
   const bool merge_small = small && !resize_target && wslots <= (uint64_t)LM_MAXS && lvl_small_on() > 1;
@@ -1289,8 +1290,8 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   } else {
     // scratch: sum of merged window sizes <= wins_bound * wslots (and <= cap + p)
     uint64_t need = a.force ? g->cap + p : wins_bound * wslots;
-    GP_CHECK(g, ensure(g->b_wk, need * 8, s));
-    GP_CHECK(g, ensure(g->b_wv, need * 4, s));
+    GP_CHECK(g, ensure(g, g->b_wk, need * 8, s));
+    GP_CHECK(g, ensure(g, g->b_wv, need * 4, s));
     a.wk = (uint64_t *)g->b_wk.p;
     a.wv = (uint32_t *)g->b_wv.p;
     a.lcnt = nullptr;
@@ -1298,10 +1299,10 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
       a.lcnt = g->cnt;                                   // the gather sums its window's leaves itself
     } else if (a.lvl) {
       uint64_t lb = wins_bound << a.lvl;
-      GP_CHECK(g, ensure(g->b_lpre, (lb + 1) * 8, s));
+      GP_CHECK(g, ensure(g, g->b_lpre, (lb + 1) * 8, s));
       a.lpre = (uint64_t *)g->b_lpre.p;
       GP_LAUNCH(g, k_lvl_leafcnt, grid_for(lb), TB, 0, s, a, g->cnt, lb);
-      scan_u64(g, a.lpre, a.lpre, lb, s);
+      GP_CHECK(g, scan_u64(g, a.lpre, a.lpre, lb, s));
     }
     uint64_t bslots = wins_bound * wslots;
     uint64_t bslots_r = (bslots + 31) & ~31ull;
@@ -1325,7 +1326,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     GP_LAUNCH(g, k_lvl_back_small, 1, LS_T, 0, s, a, g->ctrl_d);
   } else {
     GP_LAUNCH(g, k_lvl_keep, gp, TB, 0, s, a);
-    scan_u32(g, a.keep, a.kpos, p, s);
+    GP_CHECK(g, scan_u32(g, a.keep, a.kpos, p, s));
     GP_LAUNCH(g, k_lvl_summary, 1, 1, 0, s, a, g->ctrl_d);
   }
   if (g->trace_on) {
@@ -1361,21 +1362,21 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
 
 static gpma_status level_buffers(gpma *g, uint64_t n, cudaStream_t s) {
   size_t b4 = (n + 2) * 4, b8 = (n + 2) * 8;
-  GP_CHECK(g, ensure(g->b_hf, b4, s));
-  GP_CHECK(g, ensure(g->b_widx, b4, s));
-  GP_CHECK(g, ensure(g->b_wfirst, b4, s));
-  GP_CHECK(g, ensure(g->b_acc, b4, s));
-  GP_CHECK(g, ensure(g->b_aidx, b4, s));
-  GP_CHECK(g, ensure(g->b_alist, b4, s));
-  GP_CHECK(g, ensure(g->b_keep2, b4, s));
-  GP_CHECK(g, ensure(g->b_kpos, b4, s));
-  GP_CHECK(g, ensure(g->b_nw, b8, s));
-  GP_CHECK(g, ensure(g->b_woff, b8, s));
-  GP_CHECK(g, ensure(g->b_dirty, (n + 2) * sizeof(uint2), s));
+  GP_CHECK(g, ensure(g, g->b_hf, b4, s));
+  GP_CHECK(g, ensure(g, g->b_widx, b4, s));
+  GP_CHECK(g, ensure(g, g->b_wfirst, b4, s));
+  GP_CHECK(g, ensure(g, g->b_acc, b4, s));
+  GP_CHECK(g, ensure(g, g->b_aidx, b4, s));
+  GP_CHECK(g, ensure(g, g->b_alist, b4, s));
+  GP_CHECK(g, ensure(g, g->b_keep2, b4, s));
+  GP_CHECK(g, ensure(g, g->b_kpos, b4, s));
+  GP_CHECK(g, ensure(g, g->b_nw, b8, s));
+  GP_CHECK(g, ensure(g, g->b_woff, b8, s));
+  GP_CHECK(g, ensure(g, g->b_dirty, (n + 2) * sizeof(uint2), s));
   for (int i = 0; i < 2; ++i) {
-    GP_CHECK(g, ensure(g->b_pk[i], b8, s));
-    GP_CHECK(g, ensure(g->b_pv[i], b4, s));
-    GP_CHECK(g, ensure(g->b_pt[i], b4, s));
+    GP_CHECK(g, ensure(g, g->b_pk[i], b8, s));
+    GP_CHECK(g, ensure(g, g->b_pv[i], b4, s));
+    GP_CHECK(g, ensure(g, g->b_pt[i], b4, s));
   }
   return GPMA_OK;
 }
@@ -1449,10 +1450,10 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   LevelOut lo{};
   if ((st = level_step(g, a, cur, &lo, dirty_base, s, true, cap, nk, nv, ncnt))) return st;
   if (cap != g->cap) {
-    cudaFreeAsync(g->key, s);
-    cudaFreeAsync(g->val, s);
-    cudaFreeAsync(g->cnt, s);
-    cudaFreeAsync(g->head, s);
+    dev_free(g, g->key, s);
+    dev_free(g, g->val, s);
+    dev_free(g, g->cnt, s);
+    dev_free(g, g->head, s);
     g->key = nk;
     g->val = nv;
     g->cnt = ncnt;
@@ -1572,15 +1573,15 @@ __global__ void k_gather_live(const uint64_t *__restrict__ key, const uint32_t *
 static gpma_status double_root(gpma *g, cudaStream_t s) {
   gpma_status st;
   const uint64_t nl = g->cap / g->L, cap2 = g->cap * 2;
-  GP_CHECK(g, ensure(g->b_lpre, (nl + 1) * 8, s));
+  GP_CHECK(g, ensure(g, g->b_lpre, (nl + 1) * 8, s));
   uint64_t *lb = (uint64_t *)g->b_lpre.p;
   GP_LAUNCH(g, k_count_leaf_live, grid_for(nl), TB, 0, s, g->cnt, nl, lb);
-  scan_u64(g, lb, lb, nl, s);
+  GP_CHECK(g, scan_u64(g, lb, lb, nl, s));
   GP_CHECK(g, readback(g, &g->ctrl_h->sum, lb + nl, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   const uint64_t N = g->ctrl_h->sum;
-  GP_CHECK(g, ensure(g->b_wk, std::max<uint64_t>(N, 1) * 8, s));
-  GP_CHECK(g, ensure(g->b_wv, std::max<uint64_t>(N, 1) * 4, s));
+  GP_CHECK(g, ensure(g, g->b_wk, std::max<uint64_t>(N, 1) * 8, s));
+  GP_CHECK(g, ensure(g, g->b_wv, std::max<uint64_t>(N, 1) * 4, s));
   GP_LAUNCH(g, k_gather_live, grid_for(g->cap), TB, 0, s, g->key, g->val, g->L, g->cap, lb,
             (uint64_t *)g->b_wk.p, (uint32_t *)g->b_wv.p);
   uint64_t *nk;
@@ -1589,10 +1590,10 @@ static gpma_status double_root(gpma *g, cudaStream_t s) {
   if ((st = alloc_store(g, cap2, &nk, &nv, &ncnt, &nhead, s))) return st;
   GP_LAUNCH(g, k_layout_even, grid_for(cap2), TB, 0, s, (const uint64_t *)g->b_wk.p, (const uint32_t *)g->b_wv.p,
             N, nk, nv, ncnt, g->row_offset, g->L, cap2 / g->L, g->rb);
-  cudaFreeAsync(g->key, s);
-  cudaFreeAsync(g->val, s);
-  cudaFreeAsync(g->cnt, s);
-  cudaFreeAsync(g->head, s);
+  dev_free(g, g->key, s);
+  dev_free(g, g->val, s);
+  dev_free(g, g->cnt, s);
+  dev_free(g, g->head, s);
   g->key = nk;
   g->val = nv;
   g->cnt = ncnt;
@@ -1617,8 +1618,8 @@ __global__ void k_upd_summary(const uint32_t *__restrict__ pos, const uint32_t *
 // merged by the generic level step; a winner that reaches the root doubles it (l.20).
 static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
   gpma_status st;
-  GP_CHECK(g, ensure(g->b_stage[2], (p + 1) * 8, s));
-  GP_CHECK(g, ensure(g->b_stage[3], (p + 1) * 4, s));
+  GP_CHECK(g, ensure(g, g->b_stage[2], (p + 1) * 8, s));
+  GP_CHECK(g, ensure(g, g->b_stage[3], (p + 1) * 4, s));
   uint64_t *ak = (uint64_t *)g->b_stage[2].p;
   uint32_t *av = (uint32_t *)g->b_stage[3].p;
   uint64_t rounds = 0;
@@ -1632,7 +1633,7 @@ static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
     for (uint32_t lvl = 0; lvl <= g->h && nw > 0; ++lvl) {   // the root is tested too (R6)
       Lvl a = make_lvl(g, cur, nw, lvl, GPMA_INSERT);
       GP_LAUNCH(g, k_lock_winner, grid_for(nw), TB, 0, s, a.pt, nw, lvl, a.hf);
-      scan_u32(g, a.hf, a.widx, nw, s);
+      GP_CHECK(g, scan_u32(g, a.hf, a.widx, nw, s));
       GP_LAUNCH(g, k_lock_split, grid_for(nw), TB, 0, s, a.pk, a.pv, a.pt, a.hf, a.widx, nw,
                 (uint64_t *)g->b_pk[cur ^ 1].p, (uint32_t *)g->b_pv[cur ^ 1].p, (uint32_t *)g->b_pt[cur ^ 1].p, ak,
                 av, na);
@@ -1701,15 +1702,15 @@ static gpma_status upd_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, u
   if ((st = sort_unique(g, ik, op == GPMA_INSERT ? iv : nullptr, n, &m, false, which, s))) return st;
   const uint64_t *sk = (const uint64_t *)g->b_sk[*which].p;
   const uint32_t *sv = (const uint32_t *)g->b_sv[*which].p;
-  GP_CHECK(g, ensure(g->b_keep, (n + 1) * 4, s));
-  GP_CHECK(g, ensure(g->b_pos, (n + 1) * 4, s));
-  GP_CHECK(g, ensure(g->b_tgt, (n + 1) * 4, s));
+  GP_CHECK(g, ensure(g, g->b_keep, (n + 1) * 4, s));
+  GP_CHECK(g, ensure(g, g->b_pos, (n + 1) * 4, s));
+  GP_CHECK(g, ensure(g, g->b_tgt, (n + 1) * 4, s));
   if ((st = level_buffers(g, n, s))) return st;
   uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p, *tgt = (uint32_t *)g->b_tgt.p;
   GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt, g->head,
             (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb,
             g->rows_indexed ? g->row_offset : nullptr);
-  scan_u32(g, keep, pos, n, s);
+  GP_CHECK(g, scan_u32(g, keep, pos, n, s));
   GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, tgt, (uint64_t *)g->b_pk[0].p,
             (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p, g->ctrl_d);
   uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
@@ -1723,7 +1724,7 @@ static gpma_status upd_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, u
               (const uint32_t *)g->b_pv[0].p, (const uint32_t *)g->b_pt[0].p, pos + n, g->key, g->val, g->cnt,
               tmask_of(g), g->head, g->row_offset, g->rb, g->L, bound, op, keep2, (uint2 *)g->b_dirty.p,
               g->ctrl_d);
-    scan_u32(g, keep2, kpos, n, s);
+    GP_CHECK(g, scan_u32(g, keep2, kpos, n, s));
   }
   GP_LAUNCH(g, k_upd_summary, 1, 1, 0, s, pos, fused ? kpos : nullptr, n, g->ctrl_d);
   GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
@@ -1813,8 +1814,8 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   g->last = gpma_stats_t{};
   g->trace.clear();
   if (n == 0) return GPMA_OK;
-  GP_CHECK(g, ensure(g->b_stage[0], n * 8, s));
-  GP_CHECK(g, ensure(g->b_stage[1], n * 4, s));
+  GP_CHECK(g, ensure(g, g->b_stage[0], n * 8, s));
+  GP_CHECK(g, ensure(g, g->b_stage[1], n * 4, s));
   uint64_t *ik = (uint64_t *)g->b_stage[0].p;
   uint32_t *iv = (uint32_t *)g->b_stage[1].p;
   GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));

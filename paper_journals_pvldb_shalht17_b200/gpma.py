@@ -30,11 +30,34 @@ class GpmaError(RuntimeError):
         self.status = status
 
 
+ALLOC_FN = C.CFUNCTYPE(C.c_void_p, C.c_size_t, C.c_void_p, C.c_void_p)
+FREE_FN = C.CFUNCTYPE(None, C.c_void_p, C.c_void_p, C.c_void_p)
+
+
 class gpma_config(C.Structure):
     _fields_ = [("struct_size", C.c_uint32), ("leaf_slots", C.c_uint32), ("initial_capacity", C.c_uint64),
                 ("rho_leaf_bp", C.c_uint16), ("rho_root_bp", C.c_uint16), ("tau_leaf_bp", C.c_uint16),
                 ("tau_root_bp", C.c_uint16), ("init_density_bp", C.c_uint16), ("algorithm", C.c_uint16),
-                ("delete_mode", C.c_uint32), ("row_begin", C.c_uint32), ("row_end", C.c_uint32)]
+                ("delete_mode", C.c_uint32), ("row_begin", C.c_uint32), ("row_end", C.c_uint32),
+                ("alloc", ALLOC_FN), ("free", FREE_FN), ("alloc_ctx", C.c_void_p)]
+
+
+def torch_allocator_hooks():
+    """gpma_config.alloc / free through PyTorch's caching allocator (SURVEY §8(b) "Ownership":
+    the store's memory then shows up in torch.cuda.memory_allocated and is reused by torch)."""
+    import torch
+
+    def _alloc(nbytes, stream, ctx):
+        try:
+            return torch.cuda.caching_allocator_alloc(int(nbytes), stream=int(stream or 0))
+        except Exception:
+            return None          # -> GPMA_ERR_OOM
+
+    def _free(ptr, stream, ctx):
+        if ptr:
+            torch.cuda.caching_allocator_delete(int(ptr))
+
+    return ALLOC_FN(_alloc), FREE_FN(_free)
 
 
 class gpma_stats_t(C.Structure):
@@ -126,6 +149,24 @@ def _numel(a) -> int:
     return int(a.numel()) if hasattr(a, "numel") else int(a.size)
 
 
+def _itemsize(a) -> int:
+    return int(a.element_size()) if hasattr(a, "element_size") else int(a.itemsize)
+
+
+def _check_arr(a, itemsize: int, min_numel: int, what: str, device=None):
+    """Reject arrays the C ABI would read out of bounds: wrong element size, too short, or on
+    another device than the handle's (a host array is fine: the library stages it)."""
+    if a is None:
+        return
+    if _itemsize(a) != itemsize:
+        raise ValueError(f"{what}: element size {_itemsize(a)} B, expected {itemsize} B")
+    if _numel(a) < min_numel:
+        raise ValueError(f"{what}: {_numel(a)} elements, need at least {min_numel}")
+    dev = getattr(a, "device", None)
+    if device is not None and dev is not None and dev.type == "cuda" and dev.index != device:
+        raise ValueError(f"{what}: tensor on cuda:{dev.index}, handle on cuda:{device}")
+
+
 def _stream(stream):
     if stream is None:
         try:
@@ -143,17 +184,31 @@ def _stream(stream):
 class Gpma:
     """One GPMA+ store (one handle of the C ABI).  Method names follow gpma.h."""
 
-    def __init__(self, handle, num_vertices):
+    def __init__(self, handle, num_vertices, hooks=None):
         self._h = handle
         self.V = num_vertices
+        self._hooks = hooks          # keeps the allocator callbacks alive for the handle's life
+        try:
+            import torch
+            self.device = torch.cuda.current_device() if torch.cuda.is_available() else None
+        except Exception:
+            self.device = None
 
     # -- create / destroy -------------------------------------------------
     @classmethod
     def gpma_create(cls, num_vertices: int, init_keys=None, init_vals=None, *, leaf_slots: int = 0,
                     initial_capacity: int = 0, delete_mode: int = DELETE_LAZY, thresholds_bp=None,
-                    init_density_bp: int = 6000, rows=None, algorithm: int = 0, stream=None) -> "Gpma":
+                    init_density_bp: int = 6000, rows=None, algorithm: int = 0, stream=None,
+                    torch_allocator: bool = False) -> "Gpma":
         cfg = gpma_config()
         lib().gpma_config_default(C.byref(cfg))
+        hooks = None
+        if torch_allocator:
+            hooks = torch_allocator_hooks()
+            cfg.alloc, cfg.free = hooks
+        if init_keys is not None:
+            _check_arr(init_keys, 8, 0, "init_keys")
+            _check_arr(init_vals, 4, _numel(init_keys), "init_vals")
         cfg.algorithm = algorithm
         if rows is not None:
             cfg.row_begin, cfg.row_end = rows
@@ -169,7 +224,7 @@ class Gpma:
                                _stream(stream), C.byref(h))
         if st != OK:
             raise GpmaError(st, "gpma_create")
-        return cls(h, num_vertices)
+        return cls(h, num_vertices, hooks)
 
     @classmethod
     def gpma_create_raw(cls, num_vertices: int, capacity: int, leaf_slots: int, keys, vals, *,
@@ -203,6 +258,8 @@ class Gpma:
 
     # -- update -----------------------------------------------------------
     def gpma_update_batch(self, keys, vals=None, op: int = INSERT, stream=None, check: bool = True) -> int:
+        _check_arr(keys, 8, 0, "keys", self.device)
+        _check_arr(vals, 4, _numel(keys), "vals", self.device)
         st = lib().gpma_update_batch(self._h, _ptr(keys), _ptr(vals), _numel(keys), op, _stream(stream))
         if check:
             self._check(st, "gpma_update_batch")
@@ -216,16 +273,20 @@ class Gpma:
 
     # -- analytics --------------------------------------------------------
     def gpma_bfs(self, root: int, levels, stream=None):
+        _check_arr(levels, 4, self.V, "levels", self.device)
         self._check(lib().gpma_bfs(self._h, root, _ptr(levels), _stream(stream)), "gpma_bfs")
         return levels
 
     def gpma_cc(self, labels, stream=None):
+        _check_arr(labels, 4, self.V, "labels", self.device)
         self._check(lib().gpma_cc(self._h, _ptr(labels), _stream(stream)), "gpma_cc")
         return labels
 
     def gpma_pagerank(self, rank, warm_start: bool = False, damping: float = 0.85, tol_l1: float = 1e-3,
                       max_iter: int = 100, stream=None) -> int:
         it = C.c_int(0)
+        if _itemsize(rank) not in (4, 8) or _numel(rank) < self.V:
+            raise ValueError("rank: need V float64 (or float32) elements")
         f = lib().gpma_pagerank_f32 if str(getattr(rank, "dtype", "")).endswith("float32") else lib().gpma_pagerank
         self._check(f(self._h, _ptr(rank), int(warm_start), damping, tol_l1, max_iter, C.byref(it),
                       _stream(stream)), "gpma_pagerank")

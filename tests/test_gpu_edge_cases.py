@@ -108,3 +108,20 @@ def test_halving_down_to_minimum_capacity():
         _apply(g, o, [k], op=1)
     st = g.gpma_stats()
     assert st["capacity"] == o.capacity and st["live_edges"] == 0
+
+
+@pytest.mark.parametrize("n", [2047, 2048, 2049, 4095, 4096, 4097, 12289, 300_001])
+def test_sort_tiles_and_stability(n):
+    """Batch sizes around the small-sort limit (2048) and the onesweep tile (4096 keys), with
+    heavy duplication and distinct values: the stable sort must let the LAST copy of every key
+    win (R10) across tile boundaries; deletes of the same keys (keys-only sort) after that."""
+    rng = np.random.default_rng(n)
+    V = 1 << 12
+    g, o = _pair(V, [], [])
+    pool = np.unique(rng.integers(0, V, 4 * n) << 32 | rng.integers(0, V, 4 * n))[: max(n // 3, 1)]
+    keys = pool[rng.integers(0, pool.size, n)].astype(np.uint64).tolist()
+    vals = rng.integers(0, 1 << 31, n).tolist()
+    _apply(g, o, keys, vals)
+    assert_same_csr(g, o)
+    _apply(g, o, keys[: n // 2], op=1)
+    assert_same_csr(g, o)
