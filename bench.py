@@ -128,6 +128,55 @@ def algo_bytes(kernel: str, cap: int, V: int, L: int, nnz: int, dtype_bytes: int
     return None
 
 
+def update_roofline(st0: dict, st1: dict, slide_ms, B: int) -> dict:
+    """The update path against the HBM roofline (SURVEY §8(d) "Algorithmic bytes per unit of
+    work", update per batch): 12·n_ins + 8·n_del (read the batch) + Σ_W 24·|W| (read + write
+    every re-dispatched window, leaf-level absorption included) + n_del_lazy·(8L + 4) (scan
+    the leaf's keys, write the tombstone) + 8·(leaves rewritten) (heads).  Σ|W| and the key
+    counts come from the library's cumulative counters (gpma_stats.total_*) over the timed
+    slides; the time is the CUDA-event time of DELETE + INSERT of those slides."""
+    hbm, kind = peaks()
+    L = st1["leaf_slots"]
+    n_ins = st1["total_insert_keys"] - st0["total_insert_keys"]
+    n_del = st1["total_delete_keys"] - st0["total_delete_keys"]
+    slots = st1["total_slots_rewritten"] - st0["total_slots_rewritten"]
+    lazy = n_del if st1["delete_mode"] == 0 else 0
+    nb = 12 * n_ins + 8 * n_del + 24 * slots + lazy * (8 * L + 4) + 8 * (slots // L)
+    ms = float(np.sum(slide_ms))
+    ach = nb / (ms / 1e3) / 1e9
+    n = len(slide_ms)
+    return {"bound": "hbm", "achieved": ach, "peak": hbm, "unit": "GB/s", "frac": ach / hbm, "peak_kind": kind,
+            "bytes_per_slide": nb / n, "ms_per_slide": ms / n, "slots_rewritten_per_insert": slots / max(n_ins, 1),
+            "formula": "12*n_ins + 8*n_del + 24*sum|W| + n_del_lazy*(8L+4) + 8*leaves_rewritten (SURVEY 8(d))"}
+
+
+def update_kernel_table(prof: dict, st: dict, B: int) -> dict:
+    """Per-kernel times of the update path in one profiled warm step (plain launches, no graph
+    replay), with the algorithmic bytes SURVEY §8(d) assigns to the kernels that do the
+    method's data movement: lazy delete n_del·(8L+4) + 8·n_del (batch); the leaf-level merge
+    (fused level 0) 24·L per absorbed leaf + 12 per update; the existence pre-pass 12 + 8L per
+    update.  Sort / scan / compaction kernels move implementation bytes only (no frac)."""
+    hbm, _ = peaks()
+    L = st["leaf_slots"]
+    w0 = st.get("last_level0_windows", 0)
+    algo = {"k_lazy_delete": B * (8 * L + 4) + 8 * B, "k_del_mark": B * (8 * L + 4) + 8 * B,
+            "k_level0": 24 * L * w0 + 12 * B, "k_prepass": B * (12 + 8 * L)}
+    upd_names = ("k_validate", "k_lazy", "k_del", "k_prepass", "k_level0", "k_os_", "k_small_sort", "k_scan",
+                 "k_compact", "k_upd", "k_zero", "k_copy", "k_readback", "k_locate", "k_lvl", "k_heads",
+                 "k_radix")
+    out = {}
+    for k, (n, ms) in prof.items():
+        if not k.startswith(upd_names):
+            continue
+        e = {"launches": n, "ms": ms}
+        if k in algo and ms > 0:
+            e["algorithmic_bytes"] = algo[k]
+            e["achieved_gbs"] = algo[k] / (ms / 1e3) / 1e9
+            e["frac"] = e["achieved_gbs"] / hbm
+        out[k] = e
+    return dict(sorted(out.items(), key=lambda kv: -kv[1]["ms"]))
+
+
 # ------------------------------------------------------------------ GPMA arm
 def run_gpma(args, rank, world, lrank):
     from paper_journals_pvldb_shalht17_b200 import Gpma
@@ -209,6 +258,7 @@ def run_gpma(args, rank, world, lrank):
         i += 1
         prof_all = g.gpma_debug_profile_read()
         st = g.gpma_stats()
+        upd_kernels = update_kernel_table(prof_all, st, B)
         cap, L = st["capacity"], st["leaf_slots"]
         nnz = st["live_edges"]
         cand = {k: v for k, v in prof_all.items() if algo_bytes(k, cap, V, L, nnz) is not None}
@@ -216,6 +266,7 @@ def run_gpma(args, rank, world, lrank):
         evs.clear()
         pr_iters.clear()
         g.gpma_debug_profile(dom)
+        st_before = g.gpma_stats()
         launches0 = g.gpma_kernel_launches()
         if world > 1:
             torch.distributed.barrier()
@@ -251,6 +302,8 @@ def run_gpma(args, rank, world, lrank):
         iters_timed = list(pr_iters)
         st = g.gpma_stats()
         cap = st["capacity"]
+        slide_ms = phase[:, 0] + phase[:, 1]
+        upd_roof = update_roofline(st_before, st, slide_ms, B)
         # the fp32 PageRank variant on the same store (SURVEY §8(d) configs[2]: "fp64 and fp32"),
         # warm-started from the fp64 vector, outside the timed step
         x32 = x.to(torch.float32)
@@ -362,7 +415,12 @@ def run_gpma(args, rank, world, lrank):
                    "l2": "no flush: 3.2 GB store (> 126 MB L2) is streamed every step; each step reads a fresh batch"},
         "breakdown_ms": breakdown,
         "update_only": {"value": 2 * B / ((phase_ms[0] + phase_ms[1]) / 1e3), "unit": "edge updates/s",
-                        "ms_per_slide": phase_ms[0] + phase_ms[1]},
+                        "ms_per_slide": phase_ms[0] + phase_ms[1],
+                        "edges_slid_per_s": B / ((phase_ms[0] + phase_ms[1]) / 1e3),
+                        "ms_per_slide_p50": float(np.percentile(slide_ms, 50)),
+                        "ms_per_slide_p99": float(np.percentile(slide_ms, 99))},
+        "update_roofline": upd_roof,
+        "update_kernels_warm_step": upd_kernels,
         "pr_iters": iters_timed,
         "pagerank_f32": pr_f32,
         "roofline": {"bound": "hbm", "kernel": dom, "achieved": achieved, "peak": hbm, "unit": "GB/s",

@@ -111,6 +111,13 @@ typedef struct {
   uint32_t last_top_level;    /* highest level reached (h+1 = resized)                */
   uint32_t last_resized;
   uint64_t last_rounds;       /* GPMA (algorithm 1): retry rounds of the last insert    */
+  uint64_t last_level0_windows;    /* leaves rewritten at level 0 by the last batch        */
+  /* cumulative since create (measurement: SURVEY §8(d) algorithmic bytes per slide) */
+  uint64_t total_batches;     /* non-empty update batches accepted                     */
+  uint64_t total_insert_keys; /* keys of insert batches (as passed, duplicates included) */
+  uint64_t total_delete_keys; /* keys of delete batches                                */
+  uint64_t total_slots_rewritten;   /* sum of last_slots_rewritten                       */
+  uint64_t total_windows_rewritten;
 } gpma_stats_t;
 
 /* Fill *cfg with the defaults above. */

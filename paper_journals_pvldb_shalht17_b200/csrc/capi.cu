@@ -282,7 +282,14 @@ gpma_status gpma_update_batch(gpma_t *g, const uint64_t *keys, const uint32_t *v
   if (n && op == GPMA_INSERT && !vals) return GPMA_ERR_INVALID_ARG;
   if (n > 0xFFFFFFFFull) return GPMA_ERR_INVALID_ARG;
   g->st = (cudaStream_t)stream;
-  return end(g, gp::update_batch(g, keys, vals, n, (int)op, (cudaStream_t)stream));
+  st = end(g, gp::update_batch(g, keys, vals, n, (int)op, (cudaStream_t)stream));
+  if (st == GPMA_OK && n) {
+    g->tot[0] += 1;
+    g->tot[op == GPMA_INSERT ? 1 : 2] += n;
+    g->tot[3] += g->last.last_slots_rewritten;
+    g->tot[4] += g->last.last_windows_rewritten;
+  }
+  return st;
 }
 
 gpma_status gpma_bfs(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t stream) {
@@ -385,6 +392,11 @@ gpma_status gpma_stats(gpma_t *g, gpma_stats_t *out) {
   out->height = g->h;
   out->delete_mode = g->mode;
   out->resizes = g->resizes;
+  out->total_batches = g->tot[0];
+  out->total_insert_keys = g->tot[1];
+  out->total_delete_keys = g->tot[2];
+  out->total_slots_rewritten = g->tot[3];
+  out->total_windows_rewritten = g->tot[4];
   st = gp::count_slots(g, &out->live_edges, &out->tombstones, g->st);
   return end(g, st);
 }

@@ -137,6 +137,7 @@ struct gpma {
   std::atomic<uint64_t> launches{0};
   uint64_t resizes = 0;
   gpma_stats_t last{};
+  uint64_t tot[5] = {0, 0, 0, 0, 0};   // batches, insert keys, delete keys, slots, windows rewritten
   bool trace_on = false;
   std::vector<uint64_t> trace;    // (level, start, offset, flag) x4
   cudaStream_t st = nullptr;
