@@ -87,7 +87,7 @@ struct UpdGraph {
   std::vector<uint64_t> seen;     // signature after the last un-captured run of this op
   cudaGraphExec_t exec = nullptr;
   uint64_t nlaunch = 0;           // kernels in the graph (launch accounting)
-  int which = 0;                  // sort result buffer of the captured shape
+  void *srt[4] = {nullptr, nullptr, nullptr, nullptr};   // sorted batch buffers of the captured shape
 };
 
 }  // namespace gp

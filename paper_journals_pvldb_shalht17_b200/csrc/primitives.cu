@@ -675,14 +675,22 @@ __global__ void __launch_bounds__(OS_T, 2) k_os_pass(const uint64_t *__restrict_
     __threadfence();
     st[tile * 256 + t] = word;
   }
+  // windowed look-back: the words of 8 predecessors are loaded independently per round (a
+  // serial walk pays one L2 round trip per predecessor while the tiles of a wave finish)
   uint64_t excl = 0;
-  for (int64_t p = (int64_t)tile - 1; p >= 0; --p) {
-    unsigned long long x;
-    do {
-      x = st[(uint64_t)p * 256 + t];
-    } while ((x >> 62) == 0);
-    excl += x & OS_CNT_MASK;
-    if ((x >> 62) == 2) break;
+  for (int64_t p = (int64_t)tile - 1; p >= 0; p -= 8) {
+    unsigned long long x[8];
+#pragma unroll
+    for (int q = 0; q < 8; ++q) x[q] = p - q >= 0 ? st[(uint64_t)(p - q) * 256 + t] : (2ull << 62);
+    bool done = false;
+#pragma unroll
+    for (int q = 0; q < 8; ++q) {
+      if (done) break;
+      while ((x[q] >> 62) == 0) x[q] = st[(uint64_t)(p - q) * 256 + t];
+      excl += x[q] & OS_CNT_MASK;
+      done = (x[q] >> 62) == 2;
+    }
+    if (done) break;
   }
   if (tile) {
     __threadfence();

@@ -181,6 +181,295 @@ __global__ void k_lazy_delete(const uint64_t *__restrict__ keys, uint64_t n, con
   }
 }
 
+// Lazy deletion on the SORTED batch (R12): duplicates are adjacent, so only the
+// last copy of a key acts and no CAS is needed; sorted keys walk the rows (row_offset, deg) and
+// the leaves in address order, so the sectors a warp touches are shared across its lanes instead
+// of one random 32-B sector per access.  The live count / tombstone bit of a leaf and the
+// out-degree of a row are updated once per warp-run of equal leaf / row (__match_any_sync).
+__global__ void __launch_bounds__(256) k_del_mark(const uint64_t *__restrict__ sk, uint64_t n,
+                                                  const uint64_t *__restrict__ key, uint32_t *__restrict__ val,
+                                                  uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
+                                                  uint32_t nleaves, uint32_t L, uint32_t *__restrict__ tmask,
+                                                  uint32_t *__restrict__ deg, uint32_t rb, Ctrl *c,
+                                                  const uint64_t *__restrict__ ro) {
+  if (c->err) return;                                // rejected batch: nothing may change
+  const int lane = threadIdx.x & 31;
+  const uint64_t nr = (n + 31) & ~31ull;             // whole warps: the match below is full-mask
+  uint32_t marked = 0;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < nr;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    uint64_t k = KEY_NONE;
+    bool act = false;
+    if (i < n) {
+      k = sk[i];
+      act = i + 1 == n || sk[i + 1] != k;              // the last copy of a key (R10)
+    }
+    uint32_t t = 0xFFFFFFFFu, bit = 0;
+    if (act) {
+      t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
+      const uint64_t base = (uint64_t)t * L;
+      const int p = find_in_leaf(key, base, L, k);
+      if (p >= 0 && val[base + p] != VAL_TOMB) {
+        val[base + p] = VAL_TOMB;
+        bit = 1u << p;
+      } else {
+        t = 0xFFFFFFFFu;
+      }
+    }
+    const bool hit = bit != 0;
+    // per leaf: one count update and one OR of the tombstone bits
+    const uint32_t peers = __match_any_sync(0xffffffffu, t);
+    const uint32_t bits = hit ? bit : 0u;
+    uint32_t orb = bits;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {               // OR over the lanes of my leaf run
+      const uint32_t y = __shfl_xor_sync(0xffffffffu, orb, o);
+      const uint32_t peer_lane = lane ^ o;
+      if ((peers >> peer_lane) & 1u) orb |= y;
+    }
+    if (hit && lane == __ffs(peers) - 1) {
+      const uint32_t m = __popc(peers);
+      atomicSub(&cnt[t], m);
+      atomicOr(&tmask[t], orb);
+    }
+    // per row: one out-degree update
+    const uint32_t src = hit ? (uint32_t)(k >> 32) - rb : 0xFFFFFFFFu;
+    const uint32_t rp = __match_any_sync(0xffffffffu, src);
+    if (hit && lane == __ffs(rp) - 1) atomicSub(&deg[src], (uint32_t)__popc(rp));
+    marked += __popc(__ballot_sync(0xffffffffu, hit)) * (lane == 0);
+  }
+  if (lane == 0 && marked) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)marked);
+}
+
+// Target leaf of every sorted update (Alg. 4 l.3 BinarySearchLeafSegments, R9) and the head
+// flags of the leaf groups (UniqueSegments at level 0, l.18-21): a group starts where the
+// target changes.  The previous key's target comes from the neighbouring thread (shared
+// memory); only the first thread of a block searches it again.
+constexpr int LOC_T = 256;
+__global__ void __launch_bounds__(LOC_T) k_locate(const uint64_t *__restrict__ sk, uint64_t n,
+                                                  const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
+                                                  uint32_t rb, const uint64_t *__restrict__ ro,
+                                                  uint32_t *__restrict__ tgt, uint32_t *__restrict__ hf,
+                                                  const Ctrl *c) {
+  __shared__ uint32_t st[LOC_T];
+  if (c->err) return;
+  const uint64_t stride = (uint64_t)gridDim.x * LOC_T;
+  for (uint64_t b = blockIdx.x * (uint64_t)LOC_T; b < n; b += stride) {   // block-uniform
+    const uint64_t i = b + threadIdx.x;
+    uint32_t t = 0, tp = 0xFFFFFFFFu;
+    if (i < n) {
+      t = locate_leaf_rows(head, nleaves, ro, rb, L, sk[i]);
+      tgt[i] = t;
+      if (threadIdx.x == 0 && i > 0) tp = locate_leaf_rows(head, nleaves, ro, rb, L, sk[i - 1]);
+    }
+    st[threadIdx.x] = t;
+    __syncthreads();
+    if (i < n) {
+      if (threadIdx.x) tp = st[threadIdx.x - 1];
+      hf[i] = (i == 0 || tp != t) ? 1u : 0u;
+    }
+    __syncthreads();
+  }
+}
+
+__global__ void k_gstart(const uint32_t *__restrict__ hf, const uint32_t *__restrict__ gid, uint64_t n,
+                         uint32_t *__restrict__ gstart, const Ctrl *c) {
+  if (c->err) return;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    if (hf[i]) gstart[gid[i]] = (uint32_t)i;
+    if (i == 0) gstart[gid[n]] = (uint32_t)n;
+  }
+}
+
+// Fused insert pre-pass + level 0 (Alg. 4 l.3-15 at the leaves, R10-R12): one
+// L-lane sub-warp per leaf group of the sorted batch (group starts from k_gstart), the leaf
+// read ONCE.  Lane l holds slot l.  The group's updates are taken L at a time: the last copy
+// of a key acts (R10); its position among the occupied slots comes from a shuffle binary
+// search, a hit overwrites the value in place (R11) or revives a tombstone (R12), the new keys
+// are collected (shared memory) for the merge.  Density test n_live + u_new <= max_0 (R5); on
+// success the leaf is merged in registers and re-dispatched left-packed (R7 for one leaf),
+// otherwise the hits are written in place and the new keys stay pending for level 1
+// (keep[j] = 1).  Out-degrees count every new key and every revive once per row run.
+constexpr int IL_T = 256;
+__global__ void __launch_bounds__(IL_T) k_ins_leaf(const uint64_t *__restrict__ sk, const uint32_t *__restrict__ sv,
+                                                   const uint32_t *__restrict__ tgt, const uint32_t *__restrict__ gstart,
+                                                   const uint32_t *__restrict__ ng_dev, uint64_t *key, uint32_t *val,
+                                                   uint32_t *__restrict__ cnt, uint32_t *__restrict__ tmask,
+                                                   uint64_t *__restrict__ head, uint64_t *__restrict__ row_offset,
+                                                   uint32_t *__restrict__ deg, uint32_t rb, uint32_t L, uint32_t bound,
+                                                   uint32_t *__restrict__ keep, uint2 *__restrict__ dirty, Ctrl *c) {
+  __shared__ uint64_t s_nk[IL_T];                    // new keys of each sub-warp (<= L kept)
+  __shared__ uint32_t s_nv[IL_T], s_nj[IL_T];
+  __shared__ uint32_t s_hv[IL_T];                    // value a hit writes into slot l
+  if (c->err) return;
+  const uint32_t ng = *ng_dev;
+  const int lane = threadIdx.x & 31;
+  const uint32_t nsub = 32 / L, sub = lane / L, sl = lane % L;
+  const uint32_t sub0 = sub * L;                     // first lane of my sub-warp
+  const uint32_t lmask = L == 32 ? 0xffffffffu : (1u << L) - 1u;
+  const uint32_t below_me = (1u << sl) - 1u;
+  const int wb = threadIdx.x & ~31;                  // this warp's first entry in the smem arrays
+  const uint32_t lgL = __ffs(L) - 1;
+  const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  uint32_t accepted = 0, news = 0, effs = 0;
+  for (uint64_t gw = ((blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32) * nsub; gw < ng;
+       gw += nwarps * nsub) {                        // warp-uniform trip count
+    const uint64_t gi = gw + sub;
+    const bool have = gi < ng;
+    uint32_t j0 = 0, j1 = 0, t = 0;
+    if (have) {
+      j0 = gstart[gi];
+      j1 = gstart[gi + 1];
+      t = tgt[j0];
+    }
+    const uint64_t lb = (uint64_t)t * L;
+    uint64_t ks = KEY_NONE;
+    uint32_t vs = 0;
+    if (have) {
+      ks = key[lb + sl];
+      vs = val[lb + sl];
+    }
+    const bool occ = ks != KEY_NONE;
+    const uint32_t obits = (__ballot_sync(0xffffffffu, occ) >> sub0) & lmask;
+    const uint32_t nocc = __popc(obits);               // occupied prefix (sorted, left-packed)
+    const bool was_tomb = occ && vs == VAL_TOMB;
+    uint32_t hitbits = 0, nnew = 0;
+    const uint32_t u = j1 - j0;
+    const uint32_t umax = __reduce_max_sync(0xffffffffu, u);
+    for (uint32_t c0 = 0; c0 < umax; c0 += L) {        // the group's updates, L at a time
+      const uint32_t j = j0 + c0 + sl;
+      const bool inb = have && c0 + sl < u;
+      uint64_t uk = KEY_NONE;
+      uint32_t uv = 0;
+      bool eff = false;
+      if (inb) {
+        uk = sk[j];
+        uv = sv[j];
+        eff = c0 + sl + 1 == u || sk[j + 1] != uk;
+      }
+      // pos = #occupied slots with key < uk (shuffle binary search over the sorted prefix)
+      uint32_t lo = 0, hi = nocc;
+      for (uint32_t step = L; step; step >>= 1) {      // log2(L) + 1 rounds, uniform
+        const uint32_t mid = (lo + hi) >> 1;
+        const uint64_t km = __shfl_sync(0xffffffffu, ks, (int)(sub0 + (mid < L ? mid : L - 1)));
+        if (lo < hi) {
+          if (km < uk) lo = mid + 1;
+          else hi = mid;
+        }
+      }
+      const uint32_t pos = lo;
+      const uint64_t kp = __shfl_sync(0xffffffffu, ks, (int)(sub0 + (pos < L ? pos : L - 1)));
+      const uint32_t vp = __shfl_sync(0xffffffffu, vs, (int)(sub0 + (pos < L ? pos : L - 1)));
+      const bool hit = eff && pos < nocc && kp == uk;
+      if (hit) s_hv[wb + sub0 + pos] = uv;
+      const uint32_t hb = __reduce_or_sync(0xffffffffu, hit ? 1u << (sub0 + pos) : 0u);
+      hitbits |= (hb >> sub0) & lmask;
+      const bool isnew = eff && !hit;
+      const uint32_t nb = (__ballot_sync(0xffffffffu, isnew) >> sub0) & lmask;
+      if (isnew) {
+        const uint32_t q = nnew + __popc(nb & below_me);
+        if (q < L) {
+          s_nk[wb + sub0 + q] = uk;
+          s_nv[wb + sub0 + q] = uv;
+          s_nj[wb + sub0 + q] = j;
+        }
+        keep[j] = 1u;                                   // pending unless the leaf takes it
+      } else if (inb) {
+        keep[j] = 0u;
+      }
+      nnew += __popc(nb);
+      effs += eff;
+      // out-degree: every new key and every revived tombstone, once per row run
+      const bool dinc = isnew || (hit && vp == VAL_TOMB);
+      const uint32_t src = dinc ? (uint32_t)(uk >> 32) - rb : 0xFFFFFFFFu;
+      const uint32_t rp = __match_any_sync(0xffffffffu, src);
+      if (dinc && lane == __ffs(rp) - 1) atomicAdd(&deg[src], (uint32_t)__popc(rp));
+    }
+    __syncwarp();
+    news += sl == 0 ? nnew : 0;
+    const bool myhit = (hitbits >> sl) & 1u;
+    if (myhit) vs = s_hv[wb + lane];                    // overwrite (R11) / revive (R12)
+    const bool live = occ && vs != VAL_TOMB;
+    const uint32_t lbits = (__ballot_sync(0xffffffffu, live) >> sub0) & lmask;
+    const uint32_t n = __popc(lbits);
+    const bool ok = have && nnew > 0 && nnew <= bound && n + nnew <= bound;
+    // merge: a live entry's rank = its live rank + the new keys below it; a new key's rank =
+    // its index + the live entries below it (one round per new key, nnew <= max_0)
+    uint64_t uk = KEY_NONE;
+    uint32_t uv = 0;
+    if (ok && sl < nnew) {
+      uk = s_nk[wb + lane];
+      uv = s_nv[wb + lane];
+    }
+    uint32_t below_u = 0, below_l = 0;
+    const uint32_t rmax = __reduce_max_sync(0xffffffffu, ok ? nnew : 0u);
+    for (uint32_t i = 0; i < rmax; ++i) {
+      const bool vi = ok && i < nnew;
+      const uint64_t ui = __shfl_sync(0xffffffffu, uk, (int)(sub0 + (i < L ? i : 0)));
+      below_u += vi && ui < ks;
+      const uint32_t bl = __popc((__ballot_sync(0xffffffffu, vi && live && ks < ui) >> sub0) & lmask);
+      if (sl == i) below_l = bl;
+    }
+    const uint32_t N = n + nnew;
+    const uint32_t lpos = __popc(lbits & below_me) + below_u;
+    const uint32_t upos = sl + below_l;
+    const bool l0 = live && lpos == 0;
+    const bool u0 = ok && sl < nnew && upos == 0;
+    const uint32_t b0 = (__ballot_sync(0xffffffffu, l0 || u0) >> sub0) & lmask;
+    const uint64_t h_new = __shfl_sync(0xffffffffu, l0 ? ks : uk, (int)(sub0 + (b0 ? __ffs(b0) - 1 : 0)));
+    const uint64_t h_old = __shfl_sync(0xffffffffu, ks, (int)sub0);
+    __syncwarp();
+    if (ok) {
+      if (live) {
+        key[lb + lpos] = ks;
+        val[lb + lpos] = vs;
+        if (is_guard_key(ks)) row_offset[(ks >> 32) - rb + 1] = lb + lpos;
+      }
+      if (sl < nnew) {
+        key[lb + upos] = uk;
+        val[lb + upos] = uv;
+        keep[s_nj[wb + lane]] = 0u;
+      }
+    } else if (myhit) {
+      val[lb + sl] = vs;                                // in place: the leaf is not rewritten
+    }
+    __syncwarp();
+    if (ok && sl >= N) {
+      key[lb + sl] = KEY_NONE;
+      val[lb + sl] = 0;
+    }
+    const uint32_t revived = hitbits & ((__ballot_sync(0xffffffffu, was_tomb) >> sub0) & lmask);
+    if (have && sl == 0) {
+      if (ok) {
+        cnt[t] = N;
+        tmask[t] = 0u;                                  // tombstones are dropped by the rewrite
+        if (h_new != h_old && N) {
+          head[t] = h_new;
+          // empty leaves to the left carry this head (R9): leave them to the final fix-up
+          if (t > 0 && key[lb - L] == KEY_NONE) {
+            const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
+            dirty[d] = make_uint2(t, 1u);
+          }
+        }
+        ++accepted;
+      } else if (revived) {
+        cnt[t] += __popc(revived);
+        tmask[t] &= ~revived;
+      }
+    }
+    __syncwarp();
+  }
+  accepted = __reduce_add_sync(0xffffffffu, accepted);
+  news = __reduce_add_sync(0xffffffffu, news);
+  effs = __reduce_add_sync(0xffffffffu, effs);
+  if (lane == 0) {
+    if (accepted) atomicAdd((unsigned long long *)&c->windows_rewritten, (unsigned long long)accepted);
+    if (news) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)news);
+    if (effs) atomicAdd((unsigned long long *)&c->nunique, (unsigned long long)effs);
+  }
+}
+
 // Fused level 0 of the level loop (Alg. 4 l.7-15 at the leaves, where nearly every update
 // is absorbed).  A warp takes the groups of pending updates (one group per target leaf) that
 // start in its 32-item window and hands them to L-lane sub-warps (32/L groups at a time).  A
@@ -1127,25 +1416,29 @@ gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaSt
   return recompute_degrees(g, s);
 }
 
-// Sort a device batch (keys, vals) of n pairs and drop all but the last copy of each
-// key; returns the number of unique keys in *m, result in b_sk[0]/b_sv[0].
-static gpma_status sort_unique(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
-                               uint64_t *m, bool need_unique_compact, int *which, cudaStream_t s) {
-  GP_CHECK(g, ensure(g, g->b_sk[0], n * 8, s));
+// Sort a batch (Alg. 4 l.2) in place: (keys, vals) is library scratch (the staged copy of the
+// caller's batch), clobbered by the ping-pong with b_sk[1]/b_sv[1]; vals == nullptr sorts the
+// keys only.  Duplicates stay (stable: the last copy of a key is the last of its run, R10).
+struct Sorted {
+  uint64_t *k = nullptr;
+  uint32_t *v = nullptr;
+  uint64_t *ok = nullptr;      // the other buffer of the pair (free scratch after the sort)
+  uint32_t *ov = nullptr;
+};
+
+static gpma_status sort_batch(gpma *g, uint64_t *keys, uint32_t *vals, uint64_t n, Sorted *out, cudaStream_t s) {
   GP_CHECK(g, ensure(g, g->b_sk[1], n * 8, s));
-  GP_CHECK(g, ensure(g, g->b_sv[0], n * 4, s));
-  GP_CHECK(g, ensure(g, g->b_sv[1], n * 4, s));
-  uint64_t *k0 = (uint64_t *)g->b_sk[0].p, *k1 = (uint64_t *)g->b_sk[1].p;
-  uint32_t *v0 = (uint32_t *)g->b_sv[0].p, *v1 = (uint32_t *)g->b_sv[1].p;
-  GP_CHECK(g, stage_in(g, k0, keys, n * 8, s));
-  if (vals) GP_CHECK(g, stage_in(g, v0, vals, n * 4, s));
-  else GP_CHECK(g, fill_zero(g, v0, n * 4, s));
+  if (vals) GP_CHECK(g, ensure(g, g->b_sv[1], n * 4, s));
+  uint64_t *k1 = (uint64_t *)g->b_sk[1].p;
+  uint32_t *v1 = vals ? (uint32_t *)g->b_sv[1].p : nullptr;
   int sh[8];
-  int ns = key_shifts(g->V, sh);
-  GP_CHECK(g, radix_sort_pairs(g, k0, v0, k1, v1, n, sh, ns, s, which));
-  (void)need_unique_compact;
-  *m = n;
-  GP_CHECK(g, cudaGetLastError());
+  const int ns = key_shifts(g->V, sh);
+  int which = 0;
+  GP_CHECK(g, radix_sort_pairs(g, keys, vals, k1, v1, n, sh, ns, s, &which));
+  out->k = which ? k1 : keys;
+  out->v = which ? v1 : vals;
+  out->ok = which ? keys : k1;
+  out->ov = which ? vals : v1;
   return GPMA_OK;
 }
 
@@ -1175,13 +1468,10 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
     GP_CHECK(g, stage_in(g, g->b_stage[1].p, vals, n * 4, s));
     if ((st = validate(g, (uint64_t *)g->b_stage[0].p, (uint32_t *)g->b_stage[1].p, n, true, s)))
       return st;
-    int which;
-    uint64_t mm;
-    if ((st = sort_unique(g, (uint64_t *)g->b_stage[0].p, (uint32_t *)g->b_stage[1].p, n, &mm, true,
-                          &which, s)))
-      return st;
-    uint64_t *sk = (uint64_t *)g->b_sk[which].p;
-    uint32_t *sv = (uint32_t *)g->b_sv[which].p;
+    Sorted srt;
+    if ((st = sort_batch(g, (uint64_t *)g->b_stage[0].p, (uint32_t *)g->b_stage[1].p, n, &srt, s))) return st;
+    uint64_t *sk = srt.k;
+    uint32_t *sv = srt.v;
     GP_CHECK(g, ensure(g, g->b_keep, (n + 1) * 4, s));
     GP_CHECK(g, ensure(g, g->b_pos, (n + 1) * 4, s));
     uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p;
@@ -1193,8 +1483,8 @@ gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *val
     mh = (uint32_t)(g->ctrl_h->sum & 0xFFFFFFFFu);
     m = mh;
     // dense unique edges into the other buffer
-    uint64_t *uk = (uint64_t *)g->b_sk[which ^ 1].p;
-    uint32_t *uv = (uint32_t *)g->b_sv[which ^ 1].p;
+    uint64_t *uk = srt.ok;
+    uint32_t *uv = srt.ov;
     GP_LAUNCH(g, k_compact_kv, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, uk, uv);
     ek = uk;
     ev = uv;
@@ -1608,7 +1898,7 @@ static gpma_status double_root(gpma *g, cudaStream_t s) {
 
 __global__ void k_upd_summary(const uint32_t *__restrict__ pos, const uint32_t *__restrict__ kpos, uint64_t n,
                               Ctrl *c) {
-  c->sum = pos[n];                                   // pending after the pre-pass
+  if (pos) c->sum = pos[n];                          // pending after the pre-pass (else counted)
   c->sum2 = kpos ? kpos[n] : 0;                      // pending after level 0
 }
 
@@ -1663,11 +1953,10 @@ static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
                 (const uint2 *)g->b_dirty.p, dirty_base);
     }
     if (na) {                                           // the aborted insertions, sorted again
-      int which;
-      uint64_t m;
-      if ((st = sort_unique(g, ak, av, na, &m, false, &which, s))) return st;
-      GP_CHECK(g, cudaMemcpyAsync(g->b_pk[0].p, g->b_sk[which].p, na * 8, cudaMemcpyDeviceToDevice, s));
-      GP_CHECK(g, cudaMemcpyAsync(g->b_pv[0].p, g->b_sv[which].p, na * 4, cudaMemcpyDeviceToDevice, s));
+      Sorted srt;
+      if ((st = sort_batch(g, ak, av, na, &srt, s))) return st;
+      GP_CHECK(g, cudaMemcpyAsync(g->b_pk[0].p, srt.k, na * 8, cudaMemcpyDeviceToDevice, s));
+      GP_CHECK(g, cudaMemcpyAsync(g->b_pv[0].p, srt.v, na * 4, cudaMemcpyDeviceToDevice, s));
     }
     p = na;
   }
@@ -1682,38 +1971,79 @@ static gpma_status status_of(gpma *g) {
   return GPMA_OK;
 }
 
+// Strategy switches (read per call; every one is parity-tested): GPMA_DEL_SORT=0 marks lazy
+// deletes unsorted (k_lazy_delete), GPMA_INS_FUSED=0 runs the separate insert pre-pass +
+// k_level0 instead of the fused k_ins_leaf.
+static bool env_on(const char *name) {
+  const char *e = getenv(name);
+  return !e || atoi(e) != 0;
+}
+
+enum { PATH_LAZY_UNSORTED = 0, PATH_LAZY_SORTED, PATH_INS_FUSED, PATH_GENERIC };
+
+static int prefix_path(gpma *g, int op) {
+  if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) return env_on("GPMA_DEL_SORT") ? PATH_LAZY_SORTED : PATH_LAZY_UNSORTED;
+  if (op == GPMA_INSERT && g->algorithm == 0 && !g->trace_on && env_on("GPMA_INS_FUSED")) return PATH_INS_FUSED;
+  return PATH_GENERIC;
+}
+
 // The prefix of one batch, up to and including the read-back of the control block (no host
-// synchronisation inside): validate, then lazy delete, or sort -> pre-pass -> compact ->
-// fused level 0 -> summary.  *which = the sort's result buffer.
-static gpma_status upd_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int *which,
+// synchronisation inside): validate, then
+//  * lazy delete: sort the keys, mark the last copy of each (k_del_mark);
+//  * insert: sort, locate + group heads (k_locate), scan, group starts, the fused pre-pass +
+//    level 0 (k_ins_leaf), scan of the pending flags;
+//  * otherwise (strict deletes, GPMA lock-based inserts, traced batches): sort -> pre-pass ->
+//    compact -> level 0 (k_level0) unless traced -> summary.
+// *srt = the sorted batch.
+static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, int op, Sorted *srt,
                               cudaStream_t s) {
   gpma_status st;
   if ((st = zero_ctrl(g, s))) return st;
   GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, ik, iv, n, g->V, g->rb, g->nr, op == GPMA_INSERT ? 1 : 0,
             g->ctrl_d);
   const uint64_t nl = g->cap / g->L;
-  if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
+  const uint64_t *ro = g->rows_indexed ? g->row_offset : nullptr;
+  const int path = prefix_path(g, op);
+  if (path == PATH_LAZY_UNSORTED) {
     GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
-              tmask_of(g), g->deg, g->rb, g->ctrl_d, g->rows_indexed ? g->row_offset : nullptr);
+              tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
     GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
     return GPMA_OK;
   }
-  uint64_t m;
-  if ((st = sort_unique(g, ik, op == GPMA_INSERT ? iv : nullptr, n, &m, false, which, s))) return st;
-  const uint64_t *sk = (const uint64_t *)g->b_sk[*which].p;
-  const uint32_t *sv = (const uint32_t *)g->b_sv[*which].p;
+  if ((st = sort_batch(g, ik, op == GPMA_INSERT ? iv : nullptr, n, srt, s))) return st;
+  const uint64_t *sk = srt->k;
+  const uint32_t *sv = srt->v;
+  if (path == PATH_LAZY_SORTED) {
+    GP_LAUNCH(g, k_del_mark, grid_for((n + 31) / 32 * 32), 256, 0, s, sk, n, g->key, g->val, g->cnt, g->head,
+              (uint32_t)nl, g->L, tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
+    GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
+    return GPMA_OK;
+  }
   GP_CHECK(g, ensure(g, g->b_keep, (n + 1) * 4, s));
   GP_CHECK(g, ensure(g, g->b_pos, (n + 1) * 4, s));
   GP_CHECK(g, ensure(g, g->b_tgt, (n + 1) * 4, s));
   if ((st = level_buffers(g, n, s))) return st;
   uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p, *tgt = (uint32_t *)g->b_tgt.p;
+  uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
+  if (path == PATH_INS_FUSED) {
+    uint32_t *hf = keep2, *gid = kpos, *gstart = (uint32_t *)g->b_wfirst.p;
+    GP_LAUNCH(g, k_locate, grid_for(n, LOC_T), LOC_T, 0, s, sk, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tgt, hf,
+              g->ctrl_d);
+    GP_CHECK(g, scan_u32(g, hf, gid, n, s));
+    GP_LAUNCH(g, k_gstart, grid_for(n), TB, 0, s, hf, gid, n, gstart, g->ctrl_d);
+    GP_LAUNCH(g, k_ins_leaf, grid_for((n + 31) / 32 * 32, IL_T), IL_T, 0, s, sk, sv, tgt, gstart, gid + n, g->key,
+              g->val, g->cnt, tmask_of(g), g->head, g->row_offset, g->deg, g->rb, g->L, (uint32_t)g->tmax[0], keep,
+              (uint2 *)g->b_dirty.p, g->ctrl_d);
+    GP_CHECK(g, scan_u32(g, keep, pos, n, s));
+    GP_LAUNCH(g, k_upd_summary, 1, 1, 0, s, (const uint32_t *)nullptr, pos, n, g->ctrl_d);
+    GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
+    return GPMA_OK;
+  }
   GP_LAUNCH(g, k_prepass, (unsigned)((n + TB - 1) / TB), TB, 0, s, sk, sv, n, g->key, g->val, g->cnt, g->head,
-            (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb,
-            g->rows_indexed ? g->row_offset : nullptr);
+            (uint32_t)nl, g->L, op, (int)g->mode, keep, tgt, g->ctrl_d, tmask_of(g), g->deg, g->rb, ro);
   GP_CHECK(g, scan_u32(g, keep, pos, n, s));
   GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, keep, pos, n, sk, sv, tgt, (uint64_t *)g->b_pk[0].p,
             (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p, g->ctrl_d);
-  uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
   const bool lock = op == GPMA_INSERT && g->algorithm == 1;   // GPMA (Alg. 1) instead of GPMA+
   const bool fused = !g->trace_on && !lock;   // the per-level trace needs the generic level-0 step
   if (fused) {
@@ -1733,7 +2063,8 @@ static gpma_status upd_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, u
 
 // everything the prefix bakes into its launches
 static std::vector<uint64_t> upd_signature(gpma *g, uint64_t n, int op) {
-  std::vector<uint64_t> v = {n, (uint64_t)op, g->mode, g->algorithm, g->V, g->rb, g->nr, g->cap, g->L, g->h,
+  std::vector<uint64_t> v = {n, (uint64_t)op, (uint64_t)prefix_path(g, op), g->mode, g->algorithm, g->V, g->rb,
+                             g->nr, g->cap, g->L, g->h,
                              g->tmax.empty() ? 0 : g->tmax[0], g->tmin.empty() ? 0 : g->tmin[0],
                              (uint64_t)g->rows_indexed, (uint64_t)g->trace_on,
                              (uint64_t)(uintptr_t)g->key, (uint64_t)(uintptr_t)g->val, (uint64_t)(uintptr_t)g->cnt,
@@ -1777,26 +2108,29 @@ static bool upd_graph_on(gpma *g) {
 // Run the prefix: replay the cached graph when the signature matches; capture it on the second
 // run of an unchanged shape (the first run sized every buffer, so the capture allocates
 // nothing); plain launches otherwise.
-static gpma_status run_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int *which,
+static gpma_status run_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, int op, Sorted *srt,
                               cudaStream_t s) {
-  if (!s || !upd_graph_on(g)) return upd_prefix(g, ik, iv, n, op, which, s);   // (no capture on the legacy stream)
+  if (!s || !upd_graph_on(g)) return upd_prefix(g, ik, iv, n, op, srt, s);   // (no capture on the legacy stream)
   UpdGraph &G = g->ugraph[op == GPMA_INSERT ? 0 : 1];
   std::vector<uint64_t> sig = upd_signature(g, n, op);
   if (G.exec && G.sig == sig) {
     GP_CHECK(g, cudaGraphLaunch(G.exec, s));
     g->launches += G.nlaunch;
-    *which = G.which;
+    srt->k = (uint64_t *)G.srt[0];
+    srt->v = (uint32_t *)G.srt[1];
+    srt->ok = (uint64_t *)G.srt[2];
+    srt->ov = (uint32_t *)G.srt[3];
     return GPMA_OK;
   }
   if (G.seen != sig) {
-    gpma_status st = upd_prefix(g, ik, iv, n, op, which, s);
+    gpma_status st = upd_prefix(g, ik, iv, n, op, srt, s);
     G.seen = upd_signature(g, n, op);
     return st;
   }
   cudaGraph_t graph = nullptr;
   const uint64_t l0 = g->launches;
   GP_CHECK(g, cudaStreamBeginCapture(s, cudaStreamCaptureModeRelaxed));
-  gpma_status st = upd_prefix(g, ik, iv, n, op, which, s);
+  gpma_status st = upd_prefix(g, ik, iv, n, op, srt, s);
   cudaError_t e = cudaStreamEndCapture(s, &graph);
   if (st) return st;
   cudaGraphExec_t exec = nullptr;
@@ -1807,13 +2141,16 @@ static gpma_status run_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, u
     cudaGetLastError();
     g->graphs_off = true;
     g->launches = l0;
-    return upd_prefix(g, ik, iv, n, op, which, s);
+    return upd_prefix(g, ik, iv, n, op, srt, s);
   }
   if (G.exec) cudaGraphExecDestroy(G.exec);
   G.exec = exec;
   G.sig = sig;
   G.nlaunch = g->launches - l0;
-  G.which = *which;
+  G.srt[0] = srt->k;
+  G.srt[1] = srt->v;
+  G.srt[2] = srt->ok;
+  G.srt[3] = srt->ov;
   GP_CHECK(g, cudaGraphLaunch(exec, s));
   return GPMA_OK;
 }
@@ -1835,11 +2172,12 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));
   if (op == GPMA_INSERT) GP_CHECK(g, stage_in(g, iv, vals, n * 4, s));
   const uint64_t nl = g->cap / g->L;
-  int which = 0;
-  if ((st = run_prefix(g, ik, iv, n, op, &which, s))) return st;
+  const int path = prefix_path(g, op);
+  Sorted srt;
+  if ((st = run_prefix(g, ik, iv, n, op, &srt, s))) return st;
   GP_CHECK(g, cudaStreamSynchronize(s));             // the one host round trip of the batch
-  if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
-    g->last.last_unique = n;   // not deduplicated: lazy deletes are idempotent
+  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) {
+    g->last.last_unique = n;   // (lazy deletes are idempotent; the sorted path marks each key once)
     return status_of(g);
   }
   uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
@@ -1854,7 +2192,22 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   int cur = 0;
   uint64_t dirty_base = 0;
   uint32_t lvl = 0;
-  if (fused) {
+  if (path == PATH_INS_FUSED) {
+    // pending after level 0: the new keys the leaves rejected, still sorted, with their targets
+    const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
+    dirty_base = g->ctrl_h->ndirty;
+    g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;
+    g->last.last_windows_rewritten += g->ctrl_h->windows_rewritten;
+    g->last.last_level0_windows = g->ctrl_h->windows_rewritten;
+    if (p_new) {
+      GP_LAUNCH(g, k_compact_pending, grid_for(n), TB, 0, s, (const uint32_t *)g->b_keep.p,
+                (const uint32_t *)g->b_pos.p, n, srt.k, srt.v, (const uint32_t *)g->b_tgt.p, (uint64_t *)g->b_pk[0].p,
+                (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p, g->ctrl_d);
+      g->last.last_top_level = 1;
+    }
+    p = p_new;
+    lvl = 1;
+  } else if (fused) {
     const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
     dirty_base = g->ctrl_h->ndirty;
     g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;

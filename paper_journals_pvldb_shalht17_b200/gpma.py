@@ -164,7 +164,7 @@ def _check_arr(a, itemsize: int, min_numel: int, what: str, device=None):
         raise ValueError(f"{what}: element size {_itemsize(a)} B, expected {itemsize} B")
     if _numel(a) < min_numel:
         raise ValueError(f"{what}: {_numel(a)} elements, need at least {min_numel}")
-    dev = getattr(a, "device", None)
+    dev = getattr(a, "device", None) if hasattr(a, "data_ptr") else None     # torch tensors only
     if device is not None and dev is not None and dev.type == "cuda" and dev.index != device:
         raise ValueError(f"{what}: tensor on cuda:{dev.index}, handle on cuda:{device}")
 

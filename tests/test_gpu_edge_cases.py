@@ -125,3 +125,31 @@ def test_sort_tiles_and_stability(n):
     assert_same_csr(g, o)
     _apply(g, o, keys[: n // 2], op=1)
     assert_same_csr(g, o)
+
+
+def test_torch_allocator_hooks():
+    """gpma_config.alloc/free through PyTorch's caching allocator (SURVEY §8(b) "Ownership"): the
+    store lives in torch's pool while the handle lives, the results are unchanged, and destroy
+    hands every block back."""
+    from gpma_gen import config_stream
+    from paper_journals_pvldb_shalht17_b200 import Gpma
+    sw = config_stream(0, seed=9)
+    V = 1024
+    k0, v0 = sw.initial()
+    torch.cuda.synchronize()
+    before = torch.cuda.memory_allocated()
+    g = Gpma.gpma_create(V, k0.to(DEV), v0.to(DEV), torch_allocator=True)
+    o = O.Oracle(V, k0, v0)
+    cap = g.gpma_stats()["capacity"]
+    assert torch.cuda.memory_allocated() - before >= cap * 12      # keys + values at least
+    for s in range(3):
+        dk, ik, iv = sw.slide(s)
+        g.delete(dk.to(DEV))
+        g.insert(ik.to(DEV), iv.to(DEV))
+        o.delete(dk)
+        o.insert(ik, iv)
+        assert_same_layout(g, o, what=f"torch allocator slide {s}")
+    assert_same_csr(g, o)
+    g.gpma_destroy()
+    torch.cuda.synchronize()
+    assert torch.cuda.memory_allocated() == before

@@ -75,7 +75,10 @@ def test_fig5_on_gpu(golden):
     assert rp.tolist() == f5["csr_row_ptr"] and col.tolist() == f5["csr_col"]
 
 
-def _slide_parity(seed, mode, analytics=True, trace=True):
+def _slide_parity(seed, mode, analytics=True, trace=True, stream=None):
+    """One configs[0] stream, every slide.  trace=True runs the generic level-0 step (per-level
+    trace compared too); trace=False the fused kernels (k_del_mark, k_ins_leaf); a side stream
+    additionally replays the batch prefix as a CUDA graph from the second slide of a shape on."""
     sw = config_stream(0, seed=seed)
     V = 1024
     k0, v0 = sw.initial()
@@ -86,6 +89,17 @@ def _slide_parity(seed, mode, analytics=True, trace=True):
     x_g = x_o = None
     for s in range(sw.n_slides):
         dk, ik, iv = sw.slide(s)
+        if stream is not None:
+            with torch.cuda.stream(stream):
+                g.gpma_update_batch(dk.to(DEV), None, 1, stream=stream)
+                o.delete(dk)
+                assert_same_layout(g, o, what=f"seed {seed} slide {s} delete (stream)")
+                g.gpma_update_batch(ik.to(DEV), iv.to(DEV), 0, stream=stream)
+                o.insert(ik, iv)
+                stream.synchronize()
+                assert_same_layout(g, o, what=f"seed {seed} slide {s} insert (stream)")
+                assert_same_csr(g, o, what=f"seed {seed} slide {s}")
+            continue
         g.delete(dk.to(DEV))
         o.delete(dk)
         if trace and mode == DELETE_REBALANCE:
@@ -111,8 +125,30 @@ def _slide_parity(seed, mode, analytics=True, trace=True):
 
 @pytest.mark.parametrize("seed", range(20))
 def test_config0_sliding_window_lazy(seed):
-    """BASELINE configs[0]: RMAT s10 sliding window, every slide, 20 seeds."""
-    _slide_parity(seed, DELETE_LAZY)
+    """BASELINE configs[0]: RMAT s10 sliding window, every slide, 20 seeds, through
+    the fused kernels the bench times (sorted lazy delete, fused insert pre-pass + level 0)."""
+    _slide_parity(seed, DELETE_LAZY, trace=False)
+
+
+@pytest.mark.parametrize("seed", range(6))
+def test_config0_sliding_window_lazy_traced(seed):
+    """The same streams through the generic level-0 step, with the per-level trace compared."""
+    _slide_parity(seed, DELETE_LAZY, trace=True)
+
+
+@pytest.mark.parametrize("seed", range(8))
+def test_config0_sliding_window_graph_replay(seed):
+    """The 20-seed sweep's streams on a side stream: every batch after the first of a shape is a
+    replayed CUDA graph of the batch prefix (validate, sort, locate, fused leaf merge, summary)."""
+    _slide_parity(seed, DELETE_LAZY, analytics=False, trace=False, stream=torch.cuda.Stream())
+
+
+@pytest.mark.parametrize("knob", ["GPMA_DEL_SORT", "GPMA_INS_FUSED"])
+@pytest.mark.parametrize("seed", range(3))
+def test_config0_alternative_paths(seed, knob, monkeypatch):
+    """The strategy switches (unsorted lazy delete, separate pre-pass + k_level0) give the same layouts."""
+    monkeypatch.setenv(knob, "0")
+    _slide_parity(300 + seed, DELETE_LAZY, analytics=False, trace=False)
 
 
 @pytest.mark.parametrize("seed", range(5))
