@@ -182,6 +182,13 @@ gpma_status gpma_stats(gpma_t *g, gpma_stats_t *out);
 gpma_status gpma_debug_dump(gpma_t *g, uint64_t *keys, uint32_t *vals, uint64_t *row_offset,
                             uint32_t *leaf_live, uint64_t *heads, gpma_stream_t stream);
 
+/* The maintained per-leaf / per-row summaries the analytics read instead of the slots:
+ * tomb_mask u32[cap/L] (bit p = slot p of the leaf holds a tombstone, R12), leaf_guards
+ * u32[cap/L] (guards per leaf, R1), out_degree u32[row_end-row_begin] (live out-edges per
+ * owned row, PageRank's outdeg, R21).  Any output pointer may be NULL. */
+gpma_status gpma_debug_dump_aux(gpma_t *g, uint32_t *tomb_mask, uint32_t *leaf_guards, uint32_t *out_degree,
+                                gpma_stream_t stream);
+
 /* Per-level trace of the following update batches (Fig. 6 "Update Segments /
  * Offsets / Successful Flag"), off by default (it adds host syncs). */
 gpma_status gpma_debug_set_trace(gpma_t *g, int enable);
@@ -207,6 +214,43 @@ gpma_status gpma_query_neighbors(gpma_t *g, const uint32_t *verts, uint64_t n, u
  * multi-source BFS answers 64 pairs per sweep.  Unsharded stores only. */
 gpma_status gpma_query_reachable(gpma_t *g, const uint32_t *src, const uint32_t *dst, uint64_t n,
                                  uint8_t *reachable, gpma_stream_t stream);
+
+/* ---------------------------------------------------------------- multi-GPU handle
+ * SURVEY §8(b)/(e); §6.4: "We evenly partition graphs according to the vertex index
+ * and synchronize all devices after each iteration".  One process per GPU, one
+ * handle per rank; the library owns an NCCL communicator (loaded at run time: the process's
+ * libnccl.so.2, or GPMA_NCCL_LIB) and runs every exchange itself on the call's stream.
+ * Rank r's store holds the source rows [r*ceil(V/P), min(V, (r+1)*ceil(V/P))) (R24).
+ *
+ * On a handle made by gpma_dist_create, every call below is COLLECTIVE (all ranks, same order):
+ *   gpma_update_batch(keys, vals, n): the rank's slice (any n >= 0, host or device) of a global
+ *     batch; the slices are validated first and a bad key on ANY rank rejects the whole batch
+ *     on EVERY rank with the same status, nothing mutated; then routed to the owners by an
+ *     all-to-all-v in rank order (the last occurrence of a key in the global batch -- rank
+ *     order, then slice order -- wins, R10) and applied to each rank's shard.
+ *   gpma_bfs(root, levels[V]) / gpma_cc(labels[V]) / gpma_pagerank(rank[V], ...): the full,
+ *     replicated result vector on every rank (PR: fixed-point pushes reduce-scattered to their
+ *     owners each iteration, bit-identical to the single-store sums; one all-gather at the end).
+ * Local (not collective): gpma_export_csr (the owned rows: row_ptr has row_end-row_begin+1
+ * entries), gpma_stats, gpma_query_* on owned rows, gpma_destroy (collective teardown of the
+ * communicator is the caller's responsibility: destroy on every rank).  gpma_pagerank_f32 is not
+ * available on a dist handle (GPMA_ERR_INVALID_ARG). */
+
+/* 128-byte NCCL unique id (ncclGetUniqueId): call on ONE rank, broadcast it (e.g. with
+ * torch.distributed) and pass it to gpma_dist_create on every rank. */
+gpma_status gpma_dist_unique_id(void *id_out);
+
+/* Create rank `rank` of `nranks` over the global vertex set [0, num_vertices): the CUDA device
+ * current on the calling thread is the rank's GPU.  init_keys/init_vals: this rank's slice of
+ * the initial edge set (routed to the owners).  cfg: as gpma_create (row_begin/row_end are
+ * ignored -- R24 sets them).  Collective.  Errors: INVALID_ARG (nranks > V, bad rank, bad cfg),
+ * RANGE / RESERVED (a bad initial key on any rank), CUDA (NCCL missing or failing), OOM. */
+gpma_status gpma_dist_create(const void *nccl_unique_id, int rank, int nranks, uint32_t num_vertices,
+                             const uint64_t *init_keys, const uint32_t *init_vals, uint64_t n_init,
+                             const gpma_config *cfg, gpma_stream_t stream, gpma_t **out);
+
+/* Rank, rank count and owned rows of a handle (a plain handle: 0, 1, its rows). */
+gpma_status gpma_dist_info(const gpma_t *g, int *rank, int *nranks, uint32_t *row_begin, uint32_t *row_end);
 
 /* ---------------------------------------------------------------- sharded stores
  * Multi-GPU ("evenly partition graphs according to the vertex index and

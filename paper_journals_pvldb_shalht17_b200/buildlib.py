@@ -35,7 +35,7 @@ def build(force: bool = False, verbose: bool = False) -> str:
     if not force and not needs_build():
         return LIB
     os.makedirs(LIBDIR, exist_ok=True)
-    cmd = [NVCC, *ARCH, *FLAGS, "-o", LIB + ".tmp", *sources(), "-lcudart"]
+    cmd = [NVCC, *ARCH, *FLAGS, "-o", LIB + ".tmp", *sources(), "-lcudart", "-ldl"]
     if verbose:
         cmd.insert(1, "-Xptxas=-v")
     subprocess.check_call(cmd)

@@ -721,6 +721,7 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
   GP_LAUNCH(g, k_cc_compress, grid_for(V), TA, 0, s, labels, g->V);
   GP_CHECK(g, fill_zero(g, &X.ctrl_d->sum, 8, s));
   GP_LAUNCH(g, k_cc_changed, grid_for(V), TA, 0, s, labels, prev, g->V, X.ctrl_d);
+  if (!changed) return GPMA_OK;        // (changed == nullptr: the count stays in the control block)
   GP_CHECK(g, readback(g, &X.ctrl_h->sum, &X.ctrl_d->sum, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   *changed = X.ctrl_h->sum;
@@ -1098,6 +1099,7 @@ gpma_status pr_update_rows(gpma *g, double *x, const uint64_t *y_rows, double d,
   GP_CHECK(g, fill_zero(g, e_d, 8, s));
   GP_LAUNCH(g, k_prd_update_rows, grid_for(g->nr), TA, 0, s, x, (const unsigned long long *)y_rows, g->rb, g->nr,
             g->V, d, e_d);
+  if (!err) return GPMA_OK;            // (err == nullptr: the error stays in the control block, device)
   GP_CHECK(g, readback(g, &X.ctrl_h->sum2, e_d, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   memcpy(err, &X.ctrl_h->sum2, 8);

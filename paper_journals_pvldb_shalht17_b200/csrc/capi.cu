@@ -226,6 +226,61 @@ gpma_status gpma_create(uint32_t num_vertices, const uint64_t *init_keys, const 
   return GPMA_OK;
 }
 
+gpma_status gpma_dist_unique_id(void *id_out) {
+  if (!id_out) return GPMA_ERR_INVALID_ARG;
+  return gp::dist_unique_id(id_out);
+}
+
+gpma_status gpma_dist_create(const void *nccl_unique_id, int rank, int nranks, uint32_t num_vertices,
+                             const uint64_t *init_keys, const uint32_t *init_vals, uint64_t n_init,
+                             const gpma_config *cfg, gpma_stream_t stream, gpma_t **out) {
+  if (!out || !nccl_unique_id || nranks < 1 || rank < 0 || rank >= nranks || num_vertices == 0 ||
+      num_vertices == 0xFFFFFFFFu || (uint64_t)nranks > num_vertices)
+    return GPMA_ERR_INVALID_ARG;
+  if (n_init && (!init_keys || !init_vals)) return GPMA_ERR_INVALID_ARG;
+  *out = nullptr;
+  gpma *g = new_handle(num_vertices);
+  if (!g) return GPMA_ERR_OOM;
+  cudaStream_t s = (cudaStream_t)stream;
+  g->st = s;
+  gpma_config c;
+  gpma_config_default(&c);
+  if (cfg) {
+    if (cfg->struct_size < sizeof(uint32_t) * 2) {
+      free_handle(g);
+      return GPMA_ERR_INVALID_ARG;
+    }
+    memcpy(&c, cfg, cfg->struct_size < sizeof(c) ? cfg->struct_size : sizeof(c));
+  }
+  gp::dist_rows(num_vertices, nranks, rank, &c.row_begin, &c.row_end);   // R24: this rank's rows
+  uint32_t leaf = 0;
+  uint64_t cap = 0;
+  gpma_status st = apply_config(g, &c, &leaf, &cap);
+  if (st == GPMA_OK && cap && (cap & (cap - 1))) st = GPMA_ERR_INVALID_ARG;
+  if (st == GPMA_OK) st = gp::dist_attach(g, nccl_unique_id, rank, nranks);
+  if (st == GPMA_OK) st = gp::dist_create_store(g, init_keys, init_vals, n_init, cap, leaf, s);
+  if (st == GPMA_OK) {
+    cudaError_t e = cudaStreamSynchronize(s);
+    if (e) st = gp::cuda_fail(g, e, "dist_create");
+  }
+  if (st != GPMA_OK) {
+    gp::dist_detach(g);
+    free_handle(g);
+    return st;
+  }
+  *out = g;
+  return GPMA_OK;
+}
+
+gpma_status gpma_dist_info(const gpma_t *g, int *rank, int *nranks, uint32_t *row_begin, uint32_t *row_end) {
+  if (!g) return GPMA_ERR_INVALID_ARG;
+  if (rank) *rank = g->rank;
+  if (nranks) *nranks = g->nranks;
+  if (row_begin) *row_begin = g->rb;
+  if (row_end) *row_end = g->rb + g->nr;
+  return GPMA_OK;
+}
+
 gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t leaf_slots,
                             const uint64_t *keys, const uint32_t *vals, const gpma_config *cfg,
                             gpma_stream_t stream, gpma_t **out) {
@@ -269,6 +324,7 @@ gpma_status gpma_create_raw(uint32_t num_vertices, uint64_t capacity, uint32_t l
 
 gpma_status gpma_destroy(gpma_t *g) {
   if (!g) return GPMA_ERR_INVALID_ARG;
+  gp::dist_detach(g);
   free_handle(g);
   return GPMA_OK;
 }
@@ -282,7 +338,8 @@ gpma_status gpma_update_batch(gpma_t *g, const uint64_t *keys, const uint32_t *v
   if (n && op == GPMA_INSERT && !vals) return GPMA_ERR_INVALID_ARG;
   if (n > 0xFFFFFFFFull) return GPMA_ERR_INVALID_ARG;
   g->st = (cudaStream_t)stream;
-  st = end(g, gp::update_batch(g, keys, vals, n, (int)op, (cudaStream_t)stream));
+  st = end(g, g->comm ? gp::dist_update(g, keys, vals, n, (int)op, (cudaStream_t)stream)
+                      : gp::update_batch(g, keys, vals, n, (int)op, (cudaStream_t)stream));
   if (st == GPMA_OK && n) {
     g->tot[0] += 1;
     g->tot[op == GPMA_INSERT ? 1 : 2] += n;
@@ -300,7 +357,7 @@ gpma_status gpma_bfs(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t st
   Out o(g, levels, (size_t)g->V * 4, s);
   void *d;
   if (cudaError_t e = o.dev(&d, false)) return gp::cuda_fail(g, e, "bfs staging");
-  st = gp::bfs(g, root, (int32_t *)d, s);
+  st = g->comm ? gp::dist_bfs(g, root, (int32_t *)d, s) : gp::bfs(g, root, (int32_t *)d, s);
   if (st == GPMA_OK)
     if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "bfs copy-out");
   return end(g, st);
@@ -314,7 +371,7 @@ gpma_status gpma_cc(gpma_t *g, uint32_t *labels, gpma_stream_t stream) {
   Out o(g, labels, (size_t)g->V * 4, s);
   void *d;
   if (cudaError_t e = o.dev(&d, false)) return gp::cuda_fail(g, e, "cc staging");
-  st = gp::cc(g, (uint32_t *)d, s);
+  st = g->comm ? gp::dist_cc(g, (uint32_t *)d, s) : gp::cc(g, (uint32_t *)d, s);
   if (st == GPMA_OK)
     if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "cc copy-out");
   return end(g, st);
@@ -325,12 +382,13 @@ gpma_status gpma_pagerank(gpma_t *g, double *rank, int warm_start, double dampin
   gpma_status st = begin(g);
   if (st) return st;
   if (!rank || max_iter < 0 || !(damping >= 0.0 && damping <= 1.0) || !(tol_l1 >= 0.0)) return GPMA_ERR_INVALID_ARG;
-  if (g->nr != g->V) return GPMA_ERR_INVALID_ARG;   // sharded: use gpma_pr_push / gpma_pr_update
+  if (g->nr != g->V && !g->comm) return GPMA_ERR_INVALID_ARG;   // a shard driven from outside: gpma_pr_push / _update
   cudaStream_t s = (cudaStream_t)stream;
   Out o(g, rank, (size_t)g->V * 8, s);
   void *d;
   if (cudaError_t e = o.dev(&d, warm_start != 0)) return gp::cuda_fail(g, e, "pagerank staging");
-  st = gp::pagerank_f64(g, (double *)d, warm_start, damping, tol_l1, max_iter, iters_out, s);
+  st = g->comm ? gp::dist_pagerank(g, (double *)d, warm_start, damping, tol_l1, max_iter, iters_out, s)
+               : gp::pagerank_f64(g, (double *)d, warm_start, damping, tol_l1, max_iter, iters_out, s);
   if (st == GPMA_OK)
     if (cudaError_t e = o.finish()) return gp::cuda_fail(g, e, "pagerank copy-out");
   return end(g, st);
@@ -340,6 +398,7 @@ gpma_status gpma_pagerank_f32(gpma_t *g, float *rank, int warm_start, float damp
                               int *iters_out, gpma_stream_t stream) {
   gpma_status st = begin(g);
   if (st) return st;
+  if (g->comm) return GPMA_ERR_INVALID_ARG;
   if (!rank || max_iter < 0 || !(damping >= 0.0f && damping <= 1.0f) || !(tol_l1 >= 0.0f)) return GPMA_ERR_INVALID_ARG;
   if (g->nr != g->V) return GPMA_ERR_INVALID_ARG;
   cudaStream_t s = (cudaStream_t)stream;
@@ -415,6 +474,22 @@ gpma_status gpma_debug_dump(gpma_t *g, uint64_t *keys, uint32_t *vals, uint64_t 
       if (cudaError_t e = cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDefault, s))
         return gp::cuda_fail(g, e, "debug_dump");
   if (cudaError_t e = cudaStreamSynchronize(s)) return gp::cuda_fail(g, e, "debug_dump");
+  return GPMA_OK;
+}
+
+gpma_status gpma_debug_dump_aux(gpma_t *g, uint32_t *tomb_mask, uint32_t *leaf_guards, uint32_t *out_degree,
+                                gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  cudaStream_t s = (cudaStream_t)stream;
+  uint64_t nl = g->cap / g->L;
+  struct { void *dst; const void *src; size_t bytes; } cp[] = {
+      {tomb_mask, gp::tmask_of(g), nl * 4}, {leaf_guards, gp::gcnt_of(g), nl * 4}, {out_degree, g->deg, (size_t)g->nr * 4}};
+  for (auto &c : cp)
+    if (c.dst)
+      if (cudaError_t e = cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDefault, s))
+        return gp::cuda_fail(g, e, "debug_dump_aux");
+  if (cudaError_t e = cudaStreamSynchronize(s)) return gp::cuda_fail(g, e, "debug_dump_aux");
   return GPMA_OK;
 }
 

@@ -130,6 +130,11 @@ struct gpma {
   int device = 0;
   bool pool_attached = false;
 
+  // multi-GPU (gpma_dist_create, dist_nccl.cu): the rank's NCCL communicator and its scratch
+  void *comm = nullptr;           // ncclComm_t; null = a single store (or a shard driven from outside)
+  int rank = 0, nranks = 1;
+  gp::DevBuf d_k[2], d_v[2], d_misc;
+
   // state
   bool poisoned = false;
   std::string err;
@@ -233,6 +238,19 @@ gpma_status bfs_merge(gpma *g, int32_t *levels, const uint32_t *bms, uint32_t nb
 // digit shifts covering the significant bits of keys with src, dst < V
 int key_shifts(uint32_t V, int *shifts);
 
+// multi-GPU handle (dist_nccl.cu): NCCL communicator + the collective update / analytics
+void dist_rows(uint32_t V, int P, int r, uint32_t *rb, uint32_t *re);
+gpma_status dist_unique_id(void *out);
+gpma_status dist_attach(gpma *g, const void *id, int rank, int nranks);
+void dist_detach(gpma *g);
+gpma_status dist_create_store(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, uint64_t cap,
+                              uint32_t leaf, cudaStream_t s);
+gpma_status dist_update(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op, cudaStream_t s);
+gpma_status dist_bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s);
+gpma_status dist_cc(gpma *g, uint32_t *labels, cudaStream_t s);
+gpma_status dist_pagerank(gpma *g, double *x, int warm, double d, double tol, int max_iter, int *iters,
+                          cudaStream_t s);
+
 // thresholds (R4/R5) -- the library's own implementation (independent of oracle/)
 void level_bounds(uint32_t L, uint32_t h, uint32_t rho0, uint32_t rhoh, uint32_t tau0,
                   uint32_t tauh, std::vector<uint64_t> &mn, std::vector<uint64_t> &mx);
@@ -244,6 +262,10 @@ gpma_status cuda_fail(gpma *g, cudaError_t e, const char *where);
 // update engine (update.cu)
 gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op,
                          cudaStream_t s);
+gpma_status validate_slice(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, bool check_vals,
+                           cudaStream_t s);
+gpma_status create_from_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n,
+                              uint64_t cap_override, uint32_t leaf_override, cudaStream_t s);
 gpma_status build_from_sorted(gpma *g, const uint64_t *sk, const uint32_t *sv, uint64_t m,
                               cudaStream_t s);
 gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaStream_t s);

@@ -199,36 +199,34 @@ __global__ void __launch_bounds__(256) k_del_mark(const uint64_t *__restrict__ s
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < nr;
        i += (uint64_t)gridDim.x * blockDim.x) {
     uint64_t k = KEY_NONE;
-    bool act = false;
+    uint32_t t = 0xFFFFFFFFu, bit = 0;
     if (i < n) {
       k = sk[i];
-      act = i + 1 == n || sk[i + 1] != k;              // the last copy of a key (R10)
-    }
-    uint32_t t = 0xFFFFFFFFu, bit = 0;
-    if (act) {
+      // every key is located (duplicates too), so the targets of a warp are non-decreasing
+      // and lanes of one leaf form one contiguous run
       t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
-      const uint64_t base = (uint64_t)t * L;
-      const int p = find_in_leaf(key, base, L, k);
-      if (p >= 0 && val[base + p] != VAL_TOMB) {
-        val[base + p] = VAL_TOMB;
-        bit = 1u << p;
-      } else {
-        t = 0xFFFFFFFFu;
+      if (i + 1 == n || sk[i + 1] != k) {            // the last copy of a key acts (R10)
+        const uint64_t base = (uint64_t)t * L;
+        const int p = find_in_leaf(key, base, L, k);
+        if (p >= 0 && val[base + p] != VAL_TOMB) {
+          val[base + p] = VAL_TOMB;
+          bit = 1u << p;
+        }
       }
     }
     const bool hit = bit != 0;
-    // per leaf: one count update and one OR of the tombstone bits
+    // per leaf run: one count update and one OR of the tombstone bits (segmented scan)
     const uint32_t peers = __match_any_sync(0xffffffffu, t);
-    const uint32_t bits = hit ? bit : 0u;
-    uint32_t orb = bits;
+    const uint32_t hitm = __ballot_sync(0xffffffffu, hit);
+    const int first = __ffs(peers) - 1, last = 31 - __clz(peers);
+    uint32_t orb = bit;
 #pragma unroll
-    for (int o = 1; o < 32; o <<= 1) {               // OR over the lanes of my leaf run
-      const uint32_t y = __shfl_xor_sync(0xffffffffu, orb, o);
-      const uint32_t peer_lane = lane ^ o;
-      if ((peers >> peer_lane) & 1u) orb |= y;
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, orb, o);
+      if (lane - o >= first) orb |= y;
     }
-    if (hit && lane == __ffs(peers) - 1) {
-      const uint32_t m = __popc(peers);
+    const uint32_t m = __popc(peers & hitm);
+    if (lane == last && m) {
       atomicSub(&cnt[t], m);
       atomicOr(&tmask[t], orb);
     }
@@ -236,7 +234,7 @@ __global__ void __launch_bounds__(256) k_del_mark(const uint64_t *__restrict__ s
     const uint32_t src = hit ? (uint32_t)(k >> 32) - rb : 0xFFFFFFFFu;
     const uint32_t rp = __match_any_sync(0xffffffffu, src);
     if (hit && lane == __ffs(rp) - 1) atomicSub(&deg[src], (uint32_t)__popc(rp));
-    marked += __popc(__ballot_sync(0xffffffffu, hit)) * (lane == 0);
+    marked += lane == 0 ? __popc(hitm) : 0;
   }
   if (lane == 0 && marked) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)marked);
 }
@@ -1451,6 +1449,17 @@ static gpma_status validate(gpma *g, const uint64_t *keys, const uint32_t *vals,
   if ((st = read_ctrl(g, s))) return st;
   if (g->ctrl_h->err & 2u) return GPMA_ERR_RESERVED;
   if (g->ctrl_h->err & 1u) return GPMA_ERR_RANGE;
+  return GPMA_OK;
+}
+
+// Validate a caller's batch slice against the GLOBAL vertex range (multi-GPU routing runs
+// before the owner is known): ctrl.err gets the bits, no read-back (the caller reduces them).
+gpma_status validate_slice(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, bool check_vals,
+                           cudaStream_t s) {
+  gpma_status st = zero_ctrl(g, s);
+  if (st) return st;
+  if (n) GP_LAUNCH(g, k_validate, grid_for(n), TB, 0, s, keys, vals, n, g->V, 0u, g->V, check_vals ? 1 : 0, g->ctrl_d);
+  GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
 

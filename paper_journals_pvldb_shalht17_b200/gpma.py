@@ -96,6 +96,10 @@ def lib() -> C.CDLL:
             "gpma_stats": (st, [P, P]),
             "gpma_debug_dump": (st, [P, P, P, P, P, P, P]),
             "gpma_debug_set_trace": (st, [P, i32]),
+            "gpma_debug_dump_aux": (st, [P, P, P, P, P]),
+            "gpma_dist_unique_id": (st, [P]),
+            "gpma_dist_create": (st, [P, i32, i32, u32, P, P, u64, P, P, P]),
+            "gpma_dist_info": (st, [P, P, P, P, P]),
             "gpma_debug_trace": (st, [P, P, u64, P]),
             "gpma_kernel_launches": (u64, [P]),
             "gpma_route": (st, [P, P, P, u64, u32, P, P, P, P]),
@@ -128,7 +132,8 @@ EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destro
            "gpma_debug_profile", "gpma_debug_profile_read", "gpma_route", "gpma_bfs_init", "gpma_bfs_level",
            "gpma_cc_round", "gpma_pr_push", "gpma_pr_update", "gpma_pr_update_rows", "gpma_bfs_bits",
            "gpma_bfs_merge", "gpma_query_edges", "gpma_query_neighbors",
-           "gpma_query_reachable",
+           "gpma_query_reachable", "gpma_debug_dump_aux", "gpma_dist_unique_id", "gpma_dist_create",
+           "gpma_dist_info",
            "gpma_status_string", "gpma_last_error"]
 
 
@@ -310,6 +315,46 @@ class Gpma:
     def gpma_debug_dump(self, keys=None, vals=None, row_offset=None, leaf_live=None, heads=None, stream=None):
         self._check(lib().gpma_debug_dump(self._h, _ptr(keys), _ptr(vals), _ptr(row_offset), _ptr(leaf_live),
                                           _ptr(heads), _stream(stream)), "gpma_debug_dump")
+
+    def gpma_debug_dump_aux(self, tomb_mask=None, leaf_guards=None, out_degree=None, stream=None):
+        self._check(lib().gpma_debug_dump_aux(self._h, _ptr(tomb_mask), _ptr(leaf_guards), _ptr(out_degree),
+                                              _stream(stream)), "gpma_debug_dump_aux")
+
+    def gpma_dist_info(self) -> dict:
+        r, n, rb, re = C.c_int(0), C.c_int(0), C.c_uint32(0), C.c_uint32(0)
+        self._check(lib().gpma_dist_info(self._h, C.byref(r), C.byref(n), C.byref(rb), C.byref(re)), "gpma_dist_info")
+        return {"rank": r.value, "nranks": n.value, "row_begin": rb.value, "row_end": re.value}
+
+    @staticmethod
+    def gpma_dist_unique_id() -> bytes:
+        """The 128-byte NCCL unique id (call on one rank, broadcast it to the others)."""
+        buf = C.create_string_buffer(128)
+        st = lib().gpma_dist_unique_id(buf)
+        if st != OK:
+            raise GpmaError(st, "gpma_dist_unique_id (is NCCL loadable?)")
+        return buf.raw
+
+    @classmethod
+    def gpma_dist_create(cls, uid: bytes, rank: int, nranks: int, num_vertices: int, init_keys=None,
+                         init_vals=None, *, leaf_slots: int = 0, delete_mode: int = DELETE_LAZY,
+                         stream=None) -> "Gpma":
+        """Rank `rank` of a multi-GPU store (include/gpma.h "multi-GPU handle"): the library's
+        NCCL communicator runs the routing / BFS / CC / PageRank exchanges; collective."""
+        cfg = gpma_config()
+        lib().gpma_config_default(C.byref(cfg))
+        cfg.leaf_slots = leaf_slots
+        cfg.delete_mode = delete_mode
+        if init_keys is not None:
+            _check_arr(init_keys, 8, 0, "init_keys")
+            _check_arr(init_vals, 4, _numel(init_keys), "init_vals")
+        h = C.c_void_p()
+        n = 0 if init_keys is None else _numel(init_keys)
+        idb = C.create_string_buffer(bytes(uid), 128)
+        st = lib().gpma_dist_create(idb, rank, nranks, num_vertices, _ptr(init_keys), _ptr(init_vals), n,
+                                    C.byref(cfg), _stream(stream), C.byref(h))
+        if st != OK:
+            raise GpmaError(st, "gpma_dist_create")
+        return cls(h, num_vertices)
 
     def gpma_debug_set_trace(self, enable: bool):
         self._check(lib().gpma_debug_set_trace(self._h, int(enable)), "gpma_debug_set_trace")

@@ -51,7 +51,40 @@ def assert_same_layout(g, o: O.Oracle, guards=True, what=""):
     L = st["leaf_slots"]
     assert np.array_equal(gcnt, expected_leaf_live(ok, ov, L)), f"{what}: leaf live counts differ"
     assert np.array_equal(ghd, expected_heads(ok, L)), f"{what}: locate heads differ"
+    assert_same_aux(g, ok, ov, L, o.rb, o.nr, guards, what)
     return st
+
+
+def assert_same_aux(g, keys, vals, L, rb, nr, guards=True, what=""):
+    """The per-leaf tombstone masks and guard counts, and the per-row out-degrees, must be the
+    functions of the layout they summarise (they feed BFS / CC / PR / export)."""
+    nl = keys.size // L
+    tm = torch.empty(nl, dtype=torch.int32, device=DEV)
+    gc = torch.empty(nl, dtype=torch.int32, device=DEV)
+    dg = torch.empty(max(nr, 1), dtype=torch.int32, device=DEV)
+    g.gpma_debug_dump_aux(tm, gc, dg)
+    torch.cuda.synchronize()
+    tm = tm.cpu().numpy().view(np.uint32)
+    k = keys.reshape(-1, L)
+    v = vals.reshape(-1, L)
+    occ = k != KEY_NONE
+    tomb = occ & (v == np.uint32(0xFFFFFFFF))
+    want_tm = (tomb.astype(np.uint64) << np.arange(L, dtype=np.uint64)).sum(axis=1).astype(np.uint32)
+    if not np.array_equal(tm, want_tm):
+        bad = np.nonzero(tm != want_tm)[0]
+        raise AssertionError(f"{what}: tombstone masks differ at leaves {bad[:8]}: {tm[bad[:4]]} vs {want_tm[bad[:4]]}")
+    if not guards:
+        return
+    isg = occ & ((k & np.uint64(0xFFFFFFFF)) == np.uint64(0xFFFFFFFF))
+    assert np.array_equal(gc.cpu().numpy().view(np.uint32), isg.sum(axis=1).astype(np.uint32)), \
+        f"{what}: leaf guard counts differ"
+    live_edge = occ & ~isg & ~tomb
+    src = (k[live_edge] >> np.uint64(32)).astype(np.int64) - rb
+    want_deg = np.bincount(src, minlength=nr)[:nr].astype(np.uint32)
+    got_deg = dg.cpu().numpy().view(np.uint32)[:nr]
+    if not np.array_equal(got_deg, want_deg):
+        bad = np.nonzero(got_deg != want_deg)[0]
+        raise AssertionError(f"{what}: out-degrees differ at rows {bad[:8]}: {got_deg[bad[:4]]} vs {want_deg[bad[:4]]}")
 
 
 def gpu_export(g):
