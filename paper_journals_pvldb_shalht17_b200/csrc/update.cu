@@ -468,6 +468,205 @@ __global__ void __launch_bounds__(IL_T) k_ins_leaf(const uint64_t *__restrict__ 
   }
 }
 
+// Fused insert pre-pass + level 0, ONE THREAD PER LEAF GROUP (the common shape: a 2^20-key
+// batch over 2^24 leaves gives ~1 update per touched leaf).  The thread holds its leaf in
+// registers (L keys + L values, 16-B vector loads and stores, statically indexed), so a group
+// costs a handful of instructions per warp instead of a sub-warp's shuffle rounds:
+//   pass 1 over the group's updates (sorted; the last copy of a key acts, R10): a key equal to
+//     an occupied slot overwrites its value (R11) or revives a tombstone (R12); the others are new;
+//   density test n_live + u_new <= max_0 (Alg. 4 l.25, R5);
+//   accepted: tombstones dropped (left-pack by a static select network), the new keys inserted
+//     in key order (one static shift each), the leaf written back left-packed (R7 for a single
+//     leaf), count / tombstone mask / head / guard row offsets maintained;
+//   rejected: the hits written in place, the new keys flagged pending for level 1 (keep[j] = 1).
+// Out-degrees: +1 per new key and per revive (one atomic per row run of the thread).
+template <int L>
+__global__ void __launch_bounds__(256) k_ins_leaf_t(const uint64_t *__restrict__ sk, const uint32_t *__restrict__ sv,
+                                                    const uint32_t *__restrict__ tgt, const uint32_t *__restrict__ gstart,
+                                                    const uint32_t *__restrict__ ng_dev, uint64_t *key, uint32_t *val,
+                                                    uint32_t *__restrict__ cnt, uint32_t *__restrict__ tmask,
+                                                    uint64_t *__restrict__ head, uint64_t *__restrict__ row_offset,
+                                                    uint32_t *__restrict__ deg, uint32_t rb, uint32_t bound,
+                                                    uint32_t *__restrict__ keep, uint2 *__restrict__ dirty, Ctrl *c) {
+  if (c->err) return;
+  const uint32_t ng = *ng_dev;
+  uint32_t accepted = 0, news = 0, effs = 0;
+  for (uint64_t gi = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; gi < ng; gi += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t j0 = gstart[gi], j1 = gstart[gi + 1];
+    const uint32_t t = tgt[j0];
+    const uint64_t lb = (uint64_t)t * L;
+    uint64_t K[L];
+    uint32_t Vv[L];
+#pragma unroll
+    for (int p = 0; p < L; p += 2) {
+      const ulonglong2 kk = *reinterpret_cast<const ulonglong2 *>(key + lb + p);
+      K[p] = kk.x;
+      K[p + 1] = kk.y;
+    }
+#pragma unroll
+    for (int p = 0; p < L; p += 4) {
+      const uint4 vv = *reinterpret_cast<const uint4 *>(val + lb + p);
+      Vv[p] = vv.x;
+      Vv[p + 1] = vv.y;
+      Vv[p + 2] = vv.z;
+      Vv[p + 3] = vv.w;
+    }
+    uint32_t occ = 0, tomb = 0;
+#pragma unroll
+    for (int p = 0; p < L; ++p) {
+      occ |= (K[p] != KEY_NONE ? 1u : 0u) << p;
+      tomb |= (K[p] != KEY_NONE && Vv[p] == VAL_TOMB ? 1u : 0u) << p;
+    }
+    // pass 1: hits (overwrite / revive) and the count of new keys
+    uint32_t hitm = 0, revm = 0, nnew = 0;
+    uint32_t dsrc = 0xFFFFFFFFu, dcnt = 0;             // out-degree run of this thread
+    for (uint32_t j = j0; j < j1; ++j) {
+      const uint64_t uk = sk[j];
+      if (j + 1 < j1 && sk[j + 1] == uk) continue;     // not the last copy (R10)
+      ++effs;
+      const uint32_t uv = sv[j];
+      uint32_t h = 0;
+#pragma unroll
+      for (int p = 0; p < L; ++p)
+        if (K[p] == uk) {
+          h = 1u << p;
+          Vv[p] = uv;
+        }
+      const bool inc = !h || (h & tomb);               // a new key or a revived tombstone
+      hitm |= h;
+      revm |= h & tomb;
+      nnew += h ? 0u : 1u;
+      if (inc) {
+        const uint32_t src = (uint32_t)(uk >> 32) - rb;
+        if (src != dsrc) {
+          if (dcnt) atomicAdd(&deg[dsrc], dcnt);
+          dsrc = src;
+          dcnt = 0;
+        }
+        ++dcnt;
+      }
+    }
+    if (dcnt) atomicAdd(&deg[dsrc], dcnt);
+    const uint32_t live = occ & ~(tomb & ~revm);
+    const uint32_t n = __popc(live);
+    const bool ok = nnew > 0 && nnew <= bound && n + nnew <= bound;
+    news += nnew;
+    if (ok) {
+      const uint64_t h_old = K[0];
+      // drop the remaining tombstones: left-pack the live entries (static select network)
+      if (live != ((1u << n) - 1u)) {
+        uint64_t K2[L];
+        uint32_t V2[L];
+#pragma unroll
+        for (int q = 0; q < L; ++q) {
+          K2[q] = KEY_NONE;
+          V2[q] = 0;
+        }
+#pragma unroll
+        for (int p = 0; p < L; ++p) {
+          const uint32_t r = __popc(live & ((1u << p) - 1u));      // rank of slot p among the live
+#pragma unroll
+          for (int q = 0; q <= p; ++q)
+            if (((live >> p) & 1u) && r == (uint32_t)q) {
+              K2[q] = K[p];
+              V2[q] = Vv[p];
+            }
+        }
+#pragma unroll
+        for (int q = 0; q < L; ++q) {
+          K[q] = K2[q];
+          Vv[q] = V2[q];
+        }
+      }
+      // merge the new keys (sorted) into the live prefix, one static shift each
+      uint32_t N = n;
+      for (uint32_t j = j0; j < j1; ++j) {
+        const uint64_t uk = sk[j];
+        if (j + 1 < j1 && sk[j + 1] == uk) continue;
+        bool present = false;
+        uint32_t pos = 0;
+#pragma unroll
+        for (int p = 0; p < L; ++p) {
+          present |= (p < (int)N) && K[p] == uk;
+          pos += (p < (int)N) && K[p] < uk;
+        }
+        if (present) continue;                         // a hit (already applied)
+        const uint32_t uv = sv[j];
+#pragma unroll
+        for (int p = L - 1; p > 0; --p)
+          if ((uint32_t)p > pos) {
+            K[p] = K[p - 1];
+            Vv[p] = Vv[p - 1];
+          }
+#pragma unroll
+        for (int p = 0; p < L; ++p)
+          if ((uint32_t)p == pos) {
+            K[p] = uk;
+            Vv[p] = uv;
+          }
+        ++N;
+      }
+#pragma unroll
+      for (int p = 0; p < L; ++p)
+        if ((uint32_t)p >= N) {
+          K[p] = KEY_NONE;
+          Vv[p] = 0;
+        }
+#pragma unroll
+      for (int p = 0; p < L; p += 2)
+        *reinterpret_cast<ulonglong2 *>(key + lb + p) = make_ulonglong2(K[p], K[p + 1]);
+#pragma unroll
+      for (int p = 0; p < L; p += 4)
+        *reinterpret_cast<uint4 *>(val + lb + p) = make_uint4(Vv[p], Vv[p + 1], Vv[p + 2], Vv[p + 3]);
+#pragma unroll
+      for (int p = 0; p < L; ++p)
+        if (is_guard_key(K[p])) row_offset[(K[p] >> 32) - rb + 1] = lb + p;   // R8: guards that moved
+      cnt[t] = N;
+      tmask[t] = 0u;                                   // tombstones are dropped by the rewrite
+      if (K[0] != h_old) {
+        head[t] = K[0];
+        // empty leaves to the left carry this head (R9): leave them to the final fix-up
+        if (t > 0 && key[lb - L] == KEY_NONE) {
+          const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
+          dirty[d] = make_uint2(t, 1u);
+        }
+      }
+      for (uint32_t j = j0; j < j1; ++j) keep[j] = 0u;
+      ++accepted;
+    } else {
+      // rejected (or nothing new): the hits in place, the new keys pending for level 1
+      if (hitm) {
+#pragma unroll
+        for (int p = 0; p < L; ++p)
+          if ((hitm >> p) & 1u) val[lb + p] = Vv[p];
+      }
+      if (revm) {
+        cnt[t] += __popc(revm);
+        tmask[t] &= ~revm;
+      }
+      for (uint32_t j = j0; j < j1; ++j) {
+        const uint64_t uk = sk[j];
+        bool pend = false;
+        if (!(j + 1 < j1 && sk[j + 1] == uk)) {
+          bool present = false;
+#pragma unroll
+          for (int p = 0; p < L; ++p) present |= ((occ >> p) & 1u) && K[p] == uk;
+          pend = !present;
+        }
+        keep[j] = pend ? 1u : 0u;
+      }
+    }
+  }
+  accepted = __reduce_add_sync(0xffffffffu, accepted);
+  news = __reduce_add_sync(0xffffffffu, news);
+  effs = __reduce_add_sync(0xffffffffu, effs);
+  if ((threadIdx.x & 31) == 0) {
+    if (accepted) atomicAdd((unsigned long long *)&c->windows_rewritten, (unsigned long long)accepted);
+    if (news) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)news);
+    if (effs) atomicAdd((unsigned long long *)&c->nunique, (unsigned long long)effs);
+  }
+}
+
 // Fused level 0 of the level loop (Alg. 4 l.7-15 at the leaves, where nearly every update
 // is absorbed).  A warp takes the groups of pending updates (one group per target leaf) that
 // start in its 32-item window and hands them to L-lane sub-warps (32/L groups at a time).  A
@@ -614,7 +813,7 @@ __global__ void k_compact_pending(const uint32_t *__restrict__ keep, const uint3
     if (keep[i]) {
       uint32_t d = pos[i];
       ok[d] = ik[i];
-      ov[d] = iv[i];
+      ov[d] = iv ? iv[i] : 0u;                      // (a delete batch is sorted keys-only)
       ot[d] = it[i];
     }
   }
@@ -1990,6 +2189,10 @@ static bool env_on(const char *name) {
 
 enum { PATH_LAZY_UNSORTED = 0, PATH_LAZY_SORTED, PATH_INS_FUSED, PATH_GENERIC };
 
+// GPMA_INS_THREAD=0: the fused insert leaf step by L-lane sub-warps (k_ins_leaf) instead of a
+// thread per leaf group (k_ins_leaf_t, L <= 16)
+static int ins_thread_mode() { return env_on("GPMA_INS_THREAD") ? 1 : 0; }
+
 static int prefix_path(gpma *g, int op) {
   if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) return env_on("GPMA_DEL_SORT") ? PATH_LAZY_SORTED : PATH_LAZY_UNSORTED;
   if (op == GPMA_INSERT && g->algorithm == 0 && !g->trace_on && env_on("GPMA_INS_FUSED")) return PATH_INS_FUSED;
@@ -2040,9 +2243,22 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
               g->ctrl_d);
     GP_CHECK(g, scan_u32(g, hf, gid, n, s));
     GP_LAUNCH(g, k_gstart, grid_for(n), TB, 0, s, hf, gid, n, gstart, g->ctrl_d);
-    GP_LAUNCH(g, k_ins_leaf, grid_for((n + 31) / 32 * 32, IL_T), IL_T, 0, s, sk, sv, tgt, gstart, gid + n, g->key,
-              g->val, g->cnt, tmask_of(g), g->head, g->row_offset, g->deg, g->rb, g->L, (uint32_t)g->tmax[0], keep,
-              (uint2 *)g->b_dirty.p, g->ctrl_d);
+    const uint32_t bound = (uint32_t)g->tmax[0];
+    uint2 *dirty = (uint2 *)g->b_dirty.p;
+    const int per_thread = ins_thread_mode();
+    if (per_thread && g->L == 16)
+      GP_LAUNCH(g, k_ins_leaf_t<16>, grid_for(n), 256, 0, s, sk, sv, tgt, gstart, gid + n, g->key, g->val, g->cnt,
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+    else if (per_thread && g->L == 8)
+      GP_LAUNCH(g, k_ins_leaf_t<8>, grid_for(n), 256, 0, s, sk, sv, tgt, gstart, gid + n, g->key, g->val, g->cnt,
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+    else if (per_thread && g->L == 4)
+      GP_LAUNCH(g, k_ins_leaf_t<4>, grid_for(n), 256, 0, s, sk, sv, tgt, gstart, gid + n, g->key, g->val, g->cnt,
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+    else
+      GP_LAUNCH(g, k_ins_leaf, grid_for((n + 31) / 32 * 32, IL_T), IL_T, 0, s, sk, sv, tgt, gstart, gid + n, g->key,
+                g->val, g->cnt, tmask_of(g), g->head, g->row_offset, g->deg, g->rb, g->L, bound, keep, dirty,
+                g->ctrl_d);
     GP_CHECK(g, scan_u32(g, keep, pos, n, s));
     GP_LAUNCH(g, k_upd_summary, 1, 1, 0, s, (const uint32_t *)nullptr, pos, n, g->ctrl_d);
     GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));

@@ -133,3 +133,46 @@ def test_exchange_primitives_against_their_definitions():
     assert np.abs(got[lo:hi] - nx).max() <= 1e-15
     assert np.array_equal(got[:lo], x[:lo]) and np.array_equal(got[hi:], x[hi:])
     assert abs(err - np.abs(nx - x[lo:hi]).sum()) <= 1e-9
+
+
+@pytest.mark.parametrize("mode", [0, 1])
+def test_dist_handle_nccl_world_one(mode):
+    """gpma_dist_create: the library's own NCCL communicator at world size 1 -- the
+    validated routing, the collective BFS / CC / PageRank, the all-gather of x -- through the
+    C ABI, against the single-store oracle (bit-exact layout; PR scale-aware), and a batch with
+    one bad key rejected before anything mutates."""
+    from paper_journals_pvldb_shalht17_b200 import Gpma, GpmaError
+    from tests.gpu_helpers import DEV, assert_pr_close, assert_same_layout, keys_t, vals_t
+    sw = config_stream(0, seed=31 + mode)
+    V = 1024
+    k0, v0 = sw.initial()
+    uid = Gpma.gpma_dist_unique_id()
+    g = Gpma.gpma_dist_create(uid, 0, 1, V, k0.to(DEV), v0.to(DEV), delete_mode=mode)
+    assert g.gpma_dist_info() == {"rank": 0, "nranks": 1, "row_begin": 0, "row_end": V}
+    o = O.Oracle(V, k0, v0, delete_mode=mode)
+    assert_same_layout(g, o, what="dist create")
+    x = None
+    for s in range(3):
+        dk, ik, iv = sw.slide(s)
+        g.delete(dk.to(DEV))
+        g.insert(ik.to(DEV), iv.to(DEV))
+        o.delete(dk)
+        o.insert(ik, iv)
+        assert_same_layout(g, o, what=f"dist slide {s}")
+        root = bfs_root(sw, 31, s)
+        lv = torch.empty(V, dtype=torch.int32, device=DEV)
+        g.gpma_bfs(root, lv)
+        assert np.array_equal(lv.cpu().numpy(), o.bfs(root)), "dist BFS"
+        lab = torch.empty(V, dtype=torch.int32, device=DEV)
+        g.gpma_cc(lab)
+        assert np.array_equal(lab.cpu().numpy().view(np.uint32), o.cc()), "dist CC"
+        xt = torch.empty(V, dtype=torch.float64, device=DEV) if x is None else torch.from_numpy(x.copy()).to(DEV)
+        it = g.gpma_pagerank(xt, warm_start=x is not None, tol_l1=0.0, max_iter=6)
+        xo, _ = o.pagerank(x=x, tol=0.0, max_iter=6)
+        assert it == 6
+        assert_pr_close(xt.cpu().numpy(), xo, what="dist PR")
+        x = xo
+    bad = keys_t([(3 << 32) | 5, (V + 7) << 32])
+    assert g.gpma_update_batch(bad, vals_t([1, 2]), 0, check=False) == 2     # RANGE, nothing applied
+    assert_same_layout(g, o, what="after a rejected dist batch")
+    g.gpma_destroy()
