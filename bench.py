@@ -159,11 +159,13 @@ def update_kernel_table(prof: dict, st: dict, B: int) -> dict:
     hbm, _ = peaks()
     L = st["leaf_slots"]
     w0 = st.get("last_level0_windows", 0)
+    leaf = 24 * L * w0 + 12 * B       # every absorbed leaf read + written, the batch read
     algo = {"k_lazy_delete": B * (8 * L + 4) + 8 * B, "k_del_mark": B * (8 * L + 4) + 8 * B,
-            "k_level0": 24 * L * w0 + 12 * B, "k_prepass": B * (12 + 8 * L)}
+            "k_level0": leaf, "k_ins_leaf": leaf, "k_ins_leaf_t": leaf, "k_ins_leaf_u": leaf,
+            "k_prepass": B * (12 + 8 * L)}
     upd_names = ("k_validate", "k_lazy", "k_del", "k_prepass", "k_level0", "k_os_", "k_small_sort", "k_scan",
                  "k_compact", "k_upd", "k_zero", "k_copy", "k_readback", "k_locate", "k_lvl", "k_heads",
-                 "k_radix")
+                 "k_radix", "k_gflags", "k_gstart", "k_ins_leaf", "k_pend")
     out = {}
     for k, (n, ms) in prof.items():
         if not k.startswith(upd_names):

@@ -667,6 +667,284 @@ __global__ void __launch_bounds__(256) k_ins_leaf_t(const uint64_t *__restrict__
   }
 }
 
+// ---- leaf-keyed insert prefix (the default): Alg. 4 l.2-3 sort the batch so that the updates
+// of one segment are contiguous (UniqueSegments, l.18-21).  Level 0 needs exactly that grouping,
+// and R9 targets are monotone in the key, so the batch is located FIRST (unsorted, one thread per
+// key) and stably sorted by target leaf: ceil(log2 leaves / 8) radix passes of (leaf, arrival
+// index) instead of 2*ceil(log2 V / 8) passes of (key, value).  Inside a group the arrival order
+// is kept, so "the last occurrence wins" (R10) is decided in the group kernel; the key order
+// inside a leaf is rebuilt by the merge; the few updates the leaves reject are sorted by key
+// before the level loop (which works on key-sorted pending lists, l.12-15).
+__global__ void k_locate_u(const uint64_t *__restrict__ ik, uint64_t n, const uint64_t *__restrict__ head,
+                           uint32_t nleaves, uint32_t L, uint32_t rb, const uint64_t *__restrict__ ro,
+                           uint64_t *__restrict__ tk, uint32_t *__restrict__ tix, const Ctrl *c) {
+  if (c->err) return;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x) {
+    tk[i] = locate_leaf_rows(head, nleaves, ro, rb, L, ik[i]);
+    tix[i] = (uint32_t)i;
+  }
+}
+
+__global__ void k_gflags(const uint64_t *__restrict__ tk, uint64_t n, uint32_t *__restrict__ hf, const Ctrl *c) {
+  if (c->err) return;
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+       i += (uint64_t)gridDim.x * blockDim.x)
+    hf[i] = (i == 0 || tk[i] != tk[i - 1]) ? 1u : 0u;
+}
+
+// One thread per leaf group of the leaf-sorted batch (updates in arrival order): the leaf in
+// registers as in k_ins_leaf_t.  Pass 1 decides every update -- a later copy of the same key in
+// the group supersedes it (R10); a key equal to an occupied slot overwrites / revives it
+// (R11, R12); the rest are new -- and writes keep[j] = 1 for the new ones.  Accepted (density
+// n_live + u_new <= max_0): tombstones dropped, the new keys inserted at their key rank (one
+// static shift each, any order), the leaf written back; rejected: hits in place, keep stays 1.
+constexpr int ILU_T = 128;      // 4 warps: 4 x 32 leaves staged in shared memory
+template <int L>
+__global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
+                                                    const uint64_t *__restrict__ tk, const uint32_t *__restrict__ tix,
+                                                    const uint32_t *__restrict__ gstart,
+                                                    const uint32_t *__restrict__ ng_dev, uint64_t *key, uint32_t *val,
+                                                    uint32_t *__restrict__ cnt, uint32_t *__restrict__ tmask,
+                                                    uint64_t *__restrict__ head, uint64_t *__restrict__ row_offset,
+                                                    uint32_t *__restrict__ deg, uint32_t rb, uint32_t bound,
+                                                    uint32_t *__restrict__ keep, uint2 *__restrict__ dirty, Ctrl *c) {
+  // Leaf I/O is warp-cooperative: the 32 leaves of a warp's 32 groups move through shared memory
+  // in coalesced 16-B chunks (L/2 lanes per leaf for the keys, L/4 for the values), so a leaf is
+  // whole 128-B lines instead of 32 single-sector requests per load instruction.
+  constexpr int KS = L + 1;                            // padded row (u64 / u32 words)
+  __shared__ uint64_t sK[ILU_T / 32][32 * KS];
+  __shared__ uint32_t sV[ILU_T / 32][32 * KS];
+  if (c->err) return;
+  const uint32_t ng = *ng_dev;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  uint64_t *const mk = sK[w];
+  uint32_t *const mv = sV[w];
+  constexpr int KL = L / 2, KQ = 32 / KL;               // key chunks per leaf, leaves per load round
+  constexpr int VL = L / 4 > 0 ? L / 4 : 1, VQ = 32 / VL;
+  uint32_t accepted = 0, news = 0, effs = 0;
+  const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t gb = (blockIdx.x * (uint64_t)blockDim.x) + (threadIdx.x & ~31); gb < ng; gb += stride) {  // warp-uniform
+    const uint64_t gi = gb + lane;
+    const bool have = gi < ng;
+    uint32_t j0 = 0, j1 = 0, t = 0;
+    if (have) {
+      j0 = gstart[gi];
+      j1 = gstart[gi + 1];
+      t = (uint32_t)tk[j0];
+    }
+    const uint64_t lb = (uint64_t)t * L;
+    // cooperative load of the 32 leaves into shared memory
+#pragma unroll
+    for (int it = 0; it < 32 / KQ; ++it) {
+      const int q = it * KQ + lane / KL, cc = lane % KL;
+      const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+      const bool hq = __shfl_sync(0xffffffffu, have, q);
+      if (hq) {
+        const ulonglong2 kk = *reinterpret_cast<const ulonglong2 *>(key + lq + 2 * cc);
+        mk[q * KS + 2 * cc] = kk.x;
+        mk[q * KS + 2 * cc + 1] = kk.y;
+      }
+    }
+#pragma unroll
+    for (int it = 0; it < 32 / VQ; ++it) {
+      const int q = it * VQ + lane / VL, cc = lane % VL;
+      const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+      const bool hq = __shfl_sync(0xffffffffu, have, q);
+      if (hq) {
+        if (L >= 4) {
+          const uint4 vv = *reinterpret_cast<const uint4 *>(val + lq + 4 * cc);
+          mv[q * KS + 4 * cc] = vv.x;
+          mv[q * KS + 4 * cc + 1] = vv.y;
+          mv[q * KS + 4 * cc + 2] = vv.z;
+          mv[q * KS + 4 * cc + 3] = vv.w;
+        }
+      }
+    }
+    __syncwarp();
+    uint64_t K[L];
+    uint32_t Vv[L];
+#pragma unroll
+    for (int p = 0; p < L; ++p) {
+      K[p] = have ? mk[lane * KS + p] : KEY_NONE;
+      Vv[p] = have ? mv[lane * KS + p] : 0u;
+    }
+    uint32_t occ = 0, tomb = 0;
+#pragma unroll
+    for (int p = 0; p < L; ++p) {
+      occ |= (K[p] != KEY_NONE ? 1u : 0u) << p;
+      tomb |= (K[p] != KEY_NONE && Vv[p] == VAL_TOMB ? 1u : 0u) << p;
+    }
+    uint32_t hitm = 0, revm = 0, nnew = 0;
+    for (uint32_t j = j0; j < j1; ++j) {
+      const uint32_t i = tix[j];
+      const uint64_t uk = ik[i];
+      bool last = true;                                  // R10: a later copy in the group wins
+      for (uint32_t j2 = j + 1; j2 < j1 && last; ++j2) last = ik[tix[j2]] != uk;
+      uint32_t h = 0;
+      if (last) {
+        ++effs;
+        const uint32_t uv = iv[i];
+#pragma unroll
+        for (int p = 0; p < L; ++p)
+          if (K[p] == uk) {
+            h = 1u << p;
+            Vv[p] = uv;
+          }
+        hitm |= h;
+        revm |= h & tomb;
+        nnew += h ? 0u : 1u;
+        if (!h || (h & tomb)) atomicAdd(&deg[(uint32_t)(uk >> 32) - rb], 1u);   // new key or revive
+      }
+      keep[j] = (last && !h) ? 1u : 0u;
+    }
+    const uint32_t live = occ & ~(tomb & ~revm);
+    const uint32_t n = __popc(live);
+    const bool ok = have && nnew > 0 && nnew <= bound && n + nnew <= bound;
+    news += nnew;
+    if (ok) {
+      const uint64_t h_old = K[0];
+      if (live != ((1u << n) - 1u)) {                   // drop the tombstones: left-pack the live
+        uint64_t K2[L];
+        uint32_t V2[L];
+#pragma unroll
+        for (int q = 0; q < L; ++q) {
+          K2[q] = KEY_NONE;
+          V2[q] = 0;
+        }
+#pragma unroll
+        for (int p = 0; p < L; ++p) {
+          const uint32_t r = __popc(live & ((1u << p) - 1u));
+#pragma unroll
+          for (int q = 0; q <= p; ++q)
+            if (((live >> p) & 1u) && r == (uint32_t)q) {
+              K2[q] = K[p];
+              V2[q] = Vv[p];
+            }
+        }
+#pragma unroll
+        for (int q = 0; q < L; ++q) {
+          K[q] = K2[q];
+          Vv[q] = V2[q];
+        }
+      }
+      uint32_t N = n;
+      for (uint32_t j = j0; j < j1; ++j) {
+        if (!keep[j]) continue;
+        keep[j] = 0u;
+        const uint32_t i = tix[j];
+        const uint64_t uk = ik[i];
+        const uint32_t uv = iv[i];
+        uint32_t pos = 0;
+#pragma unroll
+        for (int p = 0; p < L; ++p) pos += (p < (int)N) && K[p] < uk;
+#pragma unroll
+        for (int p = L - 1; p > 0; --p)
+          if ((uint32_t)p > pos) {
+            K[p] = K[p - 1];
+            Vv[p] = Vv[p - 1];
+          }
+#pragma unroll
+        for (int p = 0; p < L; ++p)
+          if ((uint32_t)p == pos) {
+            K[p] = uk;
+            Vv[p] = uv;
+          }
+        ++N;
+      }
+#pragma unroll
+      for (int p = 0; p < L; ++p)
+        if ((uint32_t)p >= N) {
+          K[p] = KEY_NONE;
+          Vv[p] = 0;
+        }
+#pragma unroll
+      for (int p = 0; p < L; ++p) {
+        mk[lane * KS + p] = K[p];
+        mv[lane * KS + p] = Vv[p];
+        if (is_guard_key(K[p])) row_offset[(K[p] >> 32) - rb + 1] = lb + p;   // R8: guards that moved
+      }
+      cnt[t] = N;
+      tmask[t] = 0u;
+      if (K[0] != h_old) {
+        head[t] = K[0];
+        if (t > 0 && key[lb - L] == KEY_NONE) {          // empty leaves to the left carry this head
+          const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
+          dirty[d] = make_uint2(t, 1u);
+        }
+      }
+      ++accepted;
+    } else if (have) {
+      if (hitm) {
+#pragma unroll
+        for (int p = 0; p < L; ++p)
+          if ((hitm >> p) & 1u) val[lb + p] = Vv[p];
+      }
+      if (revm) {
+        cnt[t] += __popc(revm);
+        tmask[t] &= ~revm;
+      }
+    }
+    __syncwarp();
+    // cooperative store of the accepted (rewritten) leaves
+#pragma unroll
+    for (int it = 0; it < 32 / KQ; ++it) {
+      const int q = it * KQ + lane / KL, cc = lane % KL;
+      const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+      const bool oq = __shfl_sync(0xffffffffu, ok, q);
+      if (oq)
+        *reinterpret_cast<ulonglong2 *>(key + lq + 2 * cc) = make_ulonglong2(mk[q * KS + 2 * cc], mk[q * KS + 2 * cc + 1]);
+    }
+#pragma unroll
+    for (int it = 0; it < 32 / VQ; ++it) {
+      const int q = it * VQ + lane / VL, cc = lane % VL;
+      const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+      const bool oq = __shfl_sync(0xffffffffu, ok, q);
+      if (oq)
+        *reinterpret_cast<uint4 *>(val + lq + 4 * cc) =
+            make_uint4(mv[q * KS + 4 * cc], mv[q * KS + 4 * cc + 1], mv[q * KS + 4 * cc + 2], mv[q * KS + 4 * cc + 3]);
+    }
+    __syncwarp();
+  }
+  accepted = __reduce_add_sync(0xffffffffu, accepted);
+  news = __reduce_add_sync(0xffffffffu, news);
+  effs = __reduce_add_sync(0xffffffffu, effs);
+  if (lane == 0) {
+    if (accepted) atomicAdd((unsigned long long *)&c->windows_rewritten, (unsigned long long)accepted);
+    if (news) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)news);
+    if (effs) atomicAdd((unsigned long long *)&c->nunique, (unsigned long long)effs);
+  }
+}
+
+// the rejected new keys (keep[j] = 1) of the leaf-sorted batch, compacted in leaf order with
+// their targets, plus 0..p-1 (the sort of the pending keys permutes it)
+__global__ void k_pend_gather(const uint32_t *__restrict__ keep, const uint32_t *__restrict__ pos, uint64_t n,
+                              const uint32_t *__restrict__ tix, const uint64_t *__restrict__ tk,
+                              const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
+                              uint64_t *__restrict__ pk, uint32_t *__restrict__ pv, uint32_t *__restrict__ pt,
+                              uint32_t *__restrict__ seq) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < n;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    if (!keep[j]) continue;
+    const uint32_t d = pos[j], i = tix[j];
+    pk[d] = ik[i];
+    pv[d] = iv[i];
+    pt[d] = (uint32_t)tk[j];
+    seq[d] = d;
+  }
+}
+
+// pending list in key order: values and targets follow the sort's permutation
+__global__ void k_pend_permute(const uint32_t *__restrict__ perm, uint64_t p, const uint32_t *__restrict__ pv_in,
+                               const uint32_t *__restrict__ pt_in, uint32_t *__restrict__ pv, uint32_t *__restrict__ pt) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < p;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t q = perm[j];
+    pv[j] = pv_in[q];
+    pt[j] = pt_in[q];
+  }
+}
+
 // Fused level 0 of the level loop (Alg. 4 l.7-15 at the leaves, where nearly every update
 // is absorbed).  A warp takes the groups of pending updates (one group per target leaf) that
 // start in its 32-item window and hands them to L-lane sub-warps (32/L groups at a time).  A
@@ -2187,16 +2465,31 @@ static bool env_on(const char *name) {
   return !e || atoi(e) != 0;
 }
 
-enum { PATH_LAZY_UNSORTED = 0, PATH_LAZY_SORTED, PATH_INS_FUSED, PATH_GENERIC };
+enum { PATH_LAZY_UNSORTED = 0, PATH_LAZY_SORTED, PATH_INS_FUSED, PATH_INS_LEAF, PATH_GENERIC };
 
 // GPMA_INS_THREAD=0: the fused insert leaf step by L-lane sub-warps (k_ins_leaf) instead of a
 // thread per leaf group (k_ins_leaf_t, L <= 16)
 static int ins_thread_mode() { return env_on("GPMA_INS_THREAD") ? 1 : 0; }
 
+// GPMA_DEL_SORT=1: lazy deletes sorted by key first (k_del_mark) instead of marked in arrival
+// order (k_lazy_delete, default: at 1 key per ~16 leaves a sort shares no sector, it only costs);
+// GPMA_INS_LEAFSORT=0: inserts sorted by key (k_locate + k_ins_leaf[_t]) instead of located first
+// and sorted by target leaf (k_locate_u + k_ins_leaf_u, default).
 static int prefix_path(gpma *g, int op) {
-  if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) return env_on("GPMA_DEL_SORT") ? PATH_LAZY_SORTED : PATH_LAZY_UNSORTED;
-  if (op == GPMA_INSERT && g->algorithm == 0 && !g->trace_on && env_on("GPMA_INS_FUSED")) return PATH_INS_FUSED;
+  if (op == GPMA_DELETE && g->mode == GPMA_DELETE_LAZY) {
+    const char *e = getenv("GPMA_DEL_SORT");
+    return (e && atoi(e) != 0) ? PATH_LAZY_SORTED : PATH_LAZY_UNSORTED;
+  }
+  if (op == GPMA_INSERT && g->algorithm == 0 && !g->trace_on && env_on("GPMA_INS_FUSED"))
+    return (g->L <= 16 && env_on("GPMA_INS_LEAFSORT")) ? PATH_INS_LEAF : PATH_INS_FUSED;
   return PATH_GENERIC;
+}
+
+static int leaf_shifts(uint64_t nleaves, int *sh) {
+  const uint32_t bits = nleaves <= 1 ? 1 : ilog2(nleaves - 1) + 1;
+  int n = 0;
+  for (uint32_t b = 0; b < bits; b += 8) sh[n++] = (int)b;
+  return n;
 }
 
 // The prefix of one batch, up to and including the read-back of the control block (no host
@@ -2219,6 +2512,46 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
   if (path == PATH_LAZY_UNSORTED) {
     GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
               tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
+    GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
+    return GPMA_OK;
+  }
+  if (path == PATH_INS_LEAF) {
+    GP_CHECK(g, ensure(g, g->b_keep, (n + 1) * 4, s));
+    GP_CHECK(g, ensure(g, g->b_pos, (n + 1) * 4, s));
+    if ((st = level_buffers(g, n, s))) return st;
+    uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p;
+    uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
+    GP_CHECK(g, ensure(g, g->b_sk[0], n * 8, s));
+    GP_CHECK(g, ensure(g, g->b_sv[0], n * 4, s));
+    GP_CHECK(g, ensure(g, g->b_sk[1], n * 8, s));
+    GP_CHECK(g, ensure(g, g->b_sv[1], n * 4, s));
+    uint64_t *tk0 = (uint64_t *)g->b_sk[0].p, *tk1 = (uint64_t *)g->b_sk[1].p;
+    uint32_t *tx0 = (uint32_t *)g->b_sv[0].p, *tx1 = (uint32_t *)g->b_sv[1].p;
+    GP_LAUNCH(g, k_locate_u, grid_for(n), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0, tx0, g->ctrl_d);
+    int sh[8], which = 0;
+    const int ns = leaf_shifts(nl, sh);
+    GP_CHECK(g, radix_sort_pairs(g, tk0, tx0, tk1, tx1, n, sh, ns, s, &which));
+    const uint64_t *tk = which ? tk1 : tk0;
+    const uint32_t *tix = which ? tx1 : tx0;
+    srt->k = (uint64_t *)tk;
+    srt->v = (uint32_t *)tix;
+    uint32_t *hf = keep2, *gid = kpos, *gstart = (uint32_t *)g->b_wfirst.p;
+    GP_LAUNCH(g, k_gflags, grid_for(n), TB, 0, s, tk, n, hf, g->ctrl_d);
+    GP_CHECK(g, scan_u32(g, hf, gid, n, s));
+    GP_LAUNCH(g, k_gstart, grid_for(n), TB, 0, s, hf, gid, n, gstart, g->ctrl_d);
+    const uint32_t bound = (uint32_t)g->tmax[0];
+    uint2 *dirty = (uint2 *)g->b_dirty.p;
+    if (g->L == 16)
+      GP_LAUNCH(g, k_ins_leaf_u<16>, grid_for(n, ILU_T), ILU_T, 0, s, ik, iv, tk, tix, gstart, gid + n, g->key, g->val, g->cnt,
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+    else if (g->L == 8)
+      GP_LAUNCH(g, k_ins_leaf_u<8>, grid_for(n, ILU_T), ILU_T, 0, s, ik, iv, tk, tix, gstart, gid + n, g->key, g->val, g->cnt,
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+    else
+      GP_LAUNCH(g, k_ins_leaf_u<4>, grid_for(n, ILU_T), ILU_T, 0, s, ik, iv, tk, tix, gstart, gid + n, g->key, g->val, g->cnt,
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+    GP_CHECK(g, scan_u32(g, keep, pos, n, s));
+    GP_LAUNCH(g, k_upd_summary, 1, 1, 0, s, (const uint32_t *)nullptr, pos, n, g->ctrl_d);
     GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
     return GPMA_OK;
   }
@@ -2318,7 +2651,7 @@ static bool prof_sees_prefix(const std::string &f) {
   if (f == "*") return true;
   static const char *pre[] = {"k_validate", "k_lazy", "k_prepass", "k_level0", "k_os_", "k_small_sort",
                               "k_scan", "k_compact", "k_upd", "k_zero", "k_copy", "k_readback", "k_locate",
-                              "k_del"};
+                              "k_del", "k_gflags", "k_gstart", "k_ins_leaf", "k_pend"};
   for (const char *p : pre)
     if (f.find(p) != std::string::npos) return true;
   return false;
@@ -2417,7 +2750,33 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   int cur = 0;
   uint64_t dirty_base = 0;
   uint32_t lvl = 0;
-  if (path == PATH_INS_FUSED) {
+  if (path == PATH_INS_LEAF) {
+    // pending after level 0: the new keys the leaves rejected, gathered in leaf order, then put
+    // in key order (the level loop's pending lists are key-sorted, Alg. 4 l.12-15)
+    const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
+    dirty_base = g->ctrl_h->ndirty;
+    g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;
+    g->last.last_windows_rewritten += g->ctrl_h->windows_rewritten;
+    g->last.last_level0_windows = g->ctrl_h->windows_rewritten;
+    if (p_new) {
+      uint64_t *pk1 = (uint64_t *)g->b_pk[1].p;
+      uint32_t *pv1 = (uint32_t *)g->b_pv[1].p, *pt1 = (uint32_t *)g->b_pt[1].p, *seq = (uint32_t *)g->b_keep2.p;
+      GP_LAUNCH(g, k_pend_gather, grid_for(n), TB, 0, s, (const uint32_t *)g->b_keep.p, (const uint32_t *)g->b_pos.p,
+                n, (const uint32_t *)srt.v, (const uint64_t *)srt.k, ik, iv, pk1, pv1, pt1, seq);
+      int sh[8], which = 0;
+      const int ns = key_shifts(g->V, sh);
+      GP_CHECK(g, radix_sort_pairs(g, pk1, seq, (uint64_t *)g->b_sk[1].p, (uint32_t *)g->b_sv[1].p, p_new, sh, ns, s,
+                                   &which));
+      const uint64_t *pks = which ? (const uint64_t *)g->b_sk[1].p : pk1;
+      const uint32_t *perm = which ? (const uint32_t *)g->b_sv[1].p : seq;
+      GP_LAUNCH(g, k_pend_permute, grid_for(p_new), TB, 0, s, perm, p_new, pv1, pt1, (uint32_t *)g->b_pv[0].p,
+                (uint32_t *)g->b_pt[0].p);
+      GP_CHECK(g, stage_in(g, g->b_pk[0].p, pks, p_new * 8, s));
+      g->last.last_top_level = 1;
+    }
+    p = p_new;
+    lvl = 1;
+  } else if (path == PATH_INS_FUSED) {
     // pending after level 0: the new keys the leaves rejected, still sorted, with their targets
     const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
     dirty_base = g->ctrl_h->ndirty;

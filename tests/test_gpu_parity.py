@@ -143,11 +143,15 @@ def test_config0_sliding_window_graph_replay(seed):
     _slide_parity(seed, DELETE_LAZY, analytics=False, trace=False, stream=torch.cuda.Stream())
 
 
-@pytest.mark.parametrize("knob", ["GPMA_DEL_SORT", "GPMA_INS_FUSED"])
+@pytest.mark.parametrize("knob", ["GPMA_DEL_SORT=1", "GPMA_INS_FUSED=0", "GPMA_INS_LEAFSORT=0",
+                                  "GPMA_INS_LEAFSORT=0,GPMA_INS_THREAD=0"])
 @pytest.mark.parametrize("seed", range(3))
 def test_config0_alternative_paths(seed, knob, monkeypatch):
-    """The strategy switches (unsorted lazy delete, separate pre-pass + k_level0) give the same layouts."""
-    monkeypatch.setenv(knob, "0")
+    """The strategy switches (sorted lazy delete; separate pre-pass + k_level0; key-sorted fused
+    insert by a thread or a sub-warp per leaf) give the same layouts as the defaults."""
+    for kv in knob.split(","):
+        k, v = kv.split("=")
+        monkeypatch.setenv(k, v)
     _slide_parity(300 + seed, DELETE_LAZY, analytics=False, trace=False)
 
 
