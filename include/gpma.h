@@ -293,6 +293,17 @@ gpma_status gpma_pr_update(gpma_t *g, double *x, uint64_t *y, double damping, do
  * vector).  P:1215-1227. */
 gpma_status gpma_pr_update_rows(gpma_t *g, double *x, const uint64_t *y_rows, double damping, double *err,
                                 gpma_stream_t stream);
+/* gpma_pr_update_rows with the error left on the DEVICE: *err_dev (device double) += the owned
+ * rows' part of ||x'-x||_1; no host synchronisation (the caller all-reduces err_dev and reads
+ * it once per iteration). */
+gpma_status gpma_pr_update_rows_dev(gpma_t *g, double *x, const uint64_t *y_rows, double damping, double *err_dev,
+                                    gpma_stream_t stream);
+/* Validate a batch slice against the GLOBAL vertex range without touching the store (the
+ * first step of a distributed update: every rank validates its slice and the ranks agree on
+ * the status before anything is routed or applied).  Returns GPMA_OK / GPMA_ERR_RANGE /
+ * GPMA_ERR_RESERVED (insert: vals checked too; vals may be NULL for a delete). */
+gpma_status gpma_validate_batch(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, gpma_op op,
+                                gpma_stream_t stream);
 /* Multi-GPU BFS exchange ("synchronize all devices after each
  * iteration"): bitmap[ceil(V/32)] (device) := bit v set iff levels[v] == depth, i.e. this
  * rank's discoveries of the level just expanded.  Ranks all-gather their bitmaps (V/8 bytes

@@ -1092,6 +1092,14 @@ __global__ void k_prd_update_rows(double *__restrict__ x, const unsigned long lo
   if (threadIdx.x == 0 && se != 0) atomicAdd(err, se);
 }
 
+gpma_status pr_update_rows_dev(gpma *g, double *x, const uint64_t *y_rows, double d, double *err_dev,
+                              cudaStream_t s) {
+  GP_LAUNCH(g, k_prd_update_rows, grid_for(g->nr), TA, 0, s, x, (const unsigned long long *)y_rows, g->rb, g->nr,
+            g->V, d, err_dev);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 gpma_status pr_update_rows(gpma *g, double *x, const uint64_t *y_rows, double d, double *err, cudaStream_t s) {
   Scratch &X = g->an[AN_PR];
   ScanScope scan_scope_(X.scan);

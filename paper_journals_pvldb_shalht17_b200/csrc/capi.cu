@@ -663,6 +663,49 @@ gpma_status gpma_pr_update_rows(gpma_t *g, double *x, const uint64_t *y_rows, do
   return end(g, gp::pr_update_rows(g, x, y_rows, damping, err, (cudaStream_t)stream));
 }
 
+gpma_status gpma_pr_update_rows_dev(gpma_t *g, double *x, const uint64_t *y_rows, double damping, double *err_dev,
+                                    gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (!x || !y_rows || !err_dev || !(damping >= 0.0 && damping <= 1.0)) return GPMA_ERR_INVALID_ARG;
+  return end(g, gp::pr_update_rows_dev(g, x, y_rows, damping, err_dev, (cudaStream_t)stream));
+}
+
+gpma_status gpma_validate_batch(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, gpma_op op,
+                                gpma_stream_t stream) {
+  gpma_status st = begin(g);
+  if (st) return st;
+  if (op != GPMA_INSERT && op != GPMA_DELETE) return GPMA_ERR_INVALID_ARG;
+  if (n && !keys) return GPMA_ERR_INVALID_ARG;
+  if (!n) return GPMA_OK;
+  cudaStream_t s = (cudaStream_t)stream;
+  gp::DevBuf kb, vb;
+  const uint64_t *kd = keys;
+  const uint32_t *vd = op == GPMA_INSERT ? vals : nullptr;
+  // host slices are staged (the kernel reads device memory)
+  if (is_host_ptr(keys)) {
+    if (cudaError_t e = gp::ensure(g, kb, n * 8, s)) return gp::cuda_fail(g, e, "validate staging");
+    if (cudaError_t e = gp::stage_in(g, kb.p, keys, n * 8, s)) return gp::cuda_fail(g, e, "validate staging");
+    kd = (const uint64_t *)kb.p;
+  }
+  if (vd && is_host_ptr(vd)) {
+    if (cudaError_t e = gp::ensure(g, vb, n * 4, s)) return gp::cuda_fail(g, e, "validate staging");
+    if (cudaError_t e = gp::stage_in(g, vb.p, vd, n * 4, s)) return gp::cuda_fail(g, e, "validate staging");
+    vd = (const uint32_t *)vb.p;
+  }
+  st = gp::validate_slice(g, kd, vd, n, vd != nullptr, s);
+  if (st == GPMA_OK) {
+    if (cudaError_t e = gp::readback(g, g->ctrl_h, g->ctrl_d, sizeof(gp::Ctrl), s)) st = gp::cuda_fail(g, e, "validate");
+    else if (cudaError_t e2 = cudaStreamSynchronize(s)) st = gp::cuda_fail(g, e2, "validate");
+  }
+  gp::release(g, kb, s);
+  gp::release(g, vb, s);
+  if (st) return end(g, st);
+  if (g->ctrl_h->err & 2u) return GPMA_ERR_RESERVED;
+  if (g->ctrl_h->err & 1u) return GPMA_ERR_RANGE;
+  return end(g, GPMA_OK);
+}
+
 gpma_status gpma_bfs_bits(gpma_t *g, const int32_t *levels, int32_t depth, uint32_t *bitmap, gpma_stream_t stream) {
   gpma_status st = begin(g);
   if (st) return st;

@@ -233,6 +233,8 @@ gpma_status cc_round(gpma *g, uint32_t *labels, int init, uint64_t *changed, cud
 gpma_status pr_push(gpma *g, double *x, int init, uint64_t *y, cudaStream_t s);
 gpma_status pr_update(gpma *g, double *x, uint64_t *y, double d, double *err, cudaStream_t s);
 gpma_status pr_update_rows(gpma *g, double *x, const uint64_t *y_rows, double d, double *err, cudaStream_t s);
+gpma_status pr_update_rows_dev(gpma *g, double *x, const uint64_t *y_rows, double d, double *err_dev,
+                              cudaStream_t s);
 gpma_status bfs_bits(gpma *g, const int32_t *levels, int32_t depth, uint32_t *bm, cudaStream_t s);
 gpma_status bfs_merge(gpma *g, int32_t *levels, const uint32_t *bms, uint32_t nbm, int32_t depth, cudaStream_t s);
 // digit shifts covering the significant bits of keys with src, dst < V

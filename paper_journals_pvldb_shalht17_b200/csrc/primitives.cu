@@ -668,23 +668,50 @@ __global__ void __launch_bounds__(OS_T, 2) k_os_pass(const uint64_t *__restrict_
     wc[ww * 256 + t] = run;
     run += c;
   }
-  // publish the tile's aggregate for digit t, then look back for the exclusive prefix
+  // publish the tile's aggregate for digit t as early as possible (successors sum it)
   volatile unsigned long long *st = status;
   {
     const unsigned long long word = ((tile == 0 ? 2ull : 1ull) << 62) | (unsigned long long)run;
     __threadfence();
     st[tile * 256 + t] = word;
   }
-  // windowed look-back: the words of 8 predecessors are loaded independently per round (a
+  // local digit offsets inside the tile (exclusive scan of the tile counts over digits), then
+  // the tile reordered by digit in shared memory -- all before the look-back, so the keys do
+  // not occupy registers while it waits
+  {
+    uint32_t x = run;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+      if (lane >= o) x += y;
+    }
+    if (lane == 31) sbase[w] = x;
+    __syncthreads();
+    uint32_t pre = 0;
+    for (int kk = 0; kk < w; ++kk) pre += sbase[kk];
+    ldoff[t] = pre + x - run;
+  }
+  __syncthreads();
+#pragma unroll
+  for (int j = 0; j < OS_I; ++j) {
+    const uint64_t i = base + j * 32 + lane;
+    if (i < n) {
+      const uint32_t d = (uint32_t)(k[j] >> shift) & 255u;
+      const uint32_t lp = ldoff[d] + wc[w * 256 + d] + r[j];
+      sk[lp] = k[j];
+      if (HASV) sv[lp] = v[j];
+    }
+  }
+  // windowed look-back: the words of 16 predecessors are loaded independently per round (a
   // serial walk pays one L2 round trip per predecessor while the tiles of a wave finish)
   uint64_t excl = 0;
-  for (int64_t p = (int64_t)tile - 1; p >= 0; p -= 8) {
-    unsigned long long x[8];
+  for (int64_t p = (int64_t)tile - 1; p >= 0; p -= 16) {
+    unsigned long long x[16];
 #pragma unroll
-    for (int q = 0; q < 8; ++q) x[q] = p - q >= 0 ? st[(uint64_t)(p - q) * 256 + t] : (2ull << 62);
+    for (int q = 0; q < 16; ++q) x[q] = p - q >= 0 ? st[(uint64_t)(p - q) * 256 + t] : (2ull << 62);
     bool done = false;
 #pragma unroll
-    for (int q = 0; q < 8; ++q) {
+    for (int q = 0; q < 16; ++q) {
       if (done) break;
       while ((x[q] >> 62) == 0) x[q] = st[(uint64_t)(p - q) * 256 + t];
       excl += x[q] & OS_CNT_MASK;
@@ -696,34 +723,7 @@ __global__ void __launch_bounds__(OS_T, 2) k_os_pass(const uint64_t *__restrict_
     __threadfence();
     st[tile * 256 + t] = (2ull << 62) | (unsigned long long)(excl + run);
   }
-  // local digit offsets inside the tile (exclusive scan of the tile counts over digits)
-  {
-    uint32_t x = run;
-#pragma unroll
-    for (int o = 1; o < 32; o <<= 1) {
-      const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
-      if (lane >= o) x += y;
-    }
-    __syncthreads();                                 // (sbase is free again)
-    if (lane == 31) sbase[w] = x;
-    __syncthreads();
-    uint32_t pre = 0;
-    for (int kk = 0; kk < w; ++kk) pre += sbase[kk];
-    ldoff[t] = pre + x - run;
-    gofs[t] = dbase + excl;
-  }
-  __syncthreads();
-  // reorder the tile by digit in shared memory
-#pragma unroll
-  for (int j = 0; j < OS_I; ++j) {
-    const uint64_t i = base + j * 32 + lane;
-    if (i < n) {
-      const uint32_t d = (uint32_t)(k[j] >> shift) & 255u;
-      const uint32_t lp = ldoff[d] + wc[w * 256 + d] + r[j];
-      sk[lp] = k[j];
-      if (HASV) sv[lp] = v[j];
-    }
-  }
+  gofs[t] = dbase + excl;
   __syncthreads();
   // write each digit's run contiguously
   const uint32_t nt = (uint32_t)min((uint64_t)OS_TILE, n - t0);

@@ -865,7 +865,7 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
         if (is_guard_key(K[p])) row_offset[(K[p] >> 32) - rb + 1] = lb + p;   // R8: guards that moved
       }
       cnt[t] = N;
-      tmask[t] = 0u;
+      if (tomb) tmask[t] = 0u;                          // (no tombstone in the leaf: already 0)
       if (K[0] != h_old) {
         head[t] = K[0];
         if (t > 0 && key[lb - L] == KEY_NONE) {          // empty leaves to the left carry this head

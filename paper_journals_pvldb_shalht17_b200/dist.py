@@ -70,6 +70,10 @@ class CudaShard:
         counts = h.gpma_route(keys, vals, P, ok, ov, stream=self.stream)
         return ok, ov, counts
 
+    def validate(self, keys, vals, op) -> int:
+        return (self.g or self.router).gpma_validate_batch(keys, vals if op == INSERT else None, op,
+                                                           stream=self.stream)
+
     def update(self, keys, vals, op):
         self.g.gpma_update_batch(keys, vals if op == INSERT else None, op, stream=self.stream)
 
@@ -93,6 +97,10 @@ class CudaShard:
 
     def pr_update_rows(self, x, y_rows, damping) -> float:
         return self.g.gpma_pr_update_rows(x, y_rows, damping, stream=self.stream)
+
+    def pr_update_rows_dev(self, x, y_rows, damping, err_dev):
+        """err_dev (device double[1]) += the owned rows' L1 change; no host synchronisation."""
+        self.g.gpma_pr_update_rows_dev(x, y_rows, err_dev, damping, stream=self.stream)
 
     def bfs_bits(self, levels, depth, bitmap):
         self.g.gpma_bfs_bits(levels, depth, bitmap, stream=self.stream)
@@ -179,7 +187,20 @@ class DistGpma:
 
     # ---- API
     def update_batch(self, keys, vals=None, op: int = INSERT):
-        """Apply this rank's contiguous slice of a global batch (collective)."""
+        """Apply this rank's contiguous slice of a global batch (collective).  Every rank validates
+        its slice and the ranks agree on the worst status (MAX all-reduce) BEFORE anything is
+        routed or applied: a bad key anywhere rejects the batch on every rank with the same
+        GpmaError, as the single-store contract rejects the whole batch (include/gpma.h)."""
+        st = self.shard.validate(keys, vals, op) if self.P > 1 else 0
+        if self.P > 1:
+            t = torch.tensor([st], dtype=torch.int32)
+            if not self._cpu_coll:
+                t = t.to(self.shard.device)
+            dist.all_reduce(t, op=dist.ReduceOp.MAX, group=self.group)
+            st = int(t.item())
+            if st:
+                from .gpma import GpmaError
+                raise GpmaError(st, "distributed update_batch: a rank's slice was rejected (nothing applied)")
         k, v = self._exchange(keys, vals)
         self.shard.update(k, v, op)
 
@@ -250,11 +271,12 @@ class DistGpma:
             dang = y[self.V:self.V + 1].clone()
             self._all_reduce(dang, dist.ReduceOp.SUM)
             yr[hi - lo:hi - lo + 1].copy_(dang)
-            e.fill_(self.shard.pr_update_rows(x, yr, damping))
+            e.zero_()
+            self.shard.pr_update_rows_dev(x, yr, damping, e)          # the local error stays on the device
             self._all_reduce(e, dist.ReduceOp.SUM)
             y.zero_()
             it += 1
-            if float(e.item()) < tol:
+            if float(e.item()) < tol:                                 # the iteration's one host read
                 break
         # replicate x: the owned slices, back to back (the last one padded to chunk)
         xs = self.shard.vertex_array(chunk * self.P, torch.float64)

@@ -113,6 +113,8 @@ def lib() -> C.CDLL:
             "gpma_pr_update": (st, [P, P, P, C.c_double, P, P]),
             "gpma_pr_update_rows": (st, [P, P, P, C.c_double, P, P]),
             "gpma_bfs_bits": (st, [P, P, i32, P, P]),
+            "gpma_pr_update_rows_dev": (st, [P, P, P, C.c_double, P, P]),
+            "gpma_validate_batch": (st, [P, P, P, u64, i32, P]),
             "gpma_bfs_merge": (st, [P, P, P, u32, i32, P]),
             "gpma_debug_profile": (st, [P, C.c_char_p]),
             "gpma_debug_profile_read": (st, [P, C.c_char_p, C.c_size_t]),
@@ -133,7 +135,7 @@ EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destro
            "gpma_cc_round", "gpma_pr_push", "gpma_pr_update", "gpma_pr_update_rows", "gpma_bfs_bits",
            "gpma_bfs_merge", "gpma_query_edges", "gpma_query_neighbors",
            "gpma_query_reachable", "gpma_debug_dump_aux", "gpma_dist_unique_id", "gpma_dist_create",
-           "gpma_dist_info",
+           "gpma_dist_info", "gpma_pr_update_rows_dev", "gpma_validate_batch",
            "gpma_status_string", "gpma_last_error"]
 
 
@@ -433,6 +435,14 @@ class Gpma:
         self._check(lib().gpma_pr_update_rows(self._h, _ptr(x), _ptr(y_rows), damping, C.byref(e),
                                               _stream(stream)), "gpma_pr_update_rows")
         return e.value
+
+    def gpma_pr_update_rows_dev(self, x, y_rows, err_dev, damping: float = 0.85, stream=None):
+        self._check(lib().gpma_pr_update_rows_dev(self._h, _ptr(x), _ptr(y_rows), damping, _ptr(err_dev),
+                                                  _stream(stream)), "gpma_pr_update_rows_dev")
+
+    def gpma_validate_batch(self, keys, vals=None, op: int = INSERT, stream=None) -> int:
+        """Status of a batch slice against the global vertex range (no mutation): 0 / 2 / 3."""
+        return int(lib().gpma_validate_batch(self._h, _ptr(keys), _ptr(vals), _numel(keys), op, _stream(stream)))
 
     def gpma_bfs_bits(self, levels, depth: int, bitmap, stream=None):
         self._check(lib().gpma_bfs_bits(self._h, _ptr(levels), depth, _ptr(bitmap), _stream(stream)),

@@ -33,6 +33,16 @@ class OracleShard:
         counts = [int((owner == r).sum()) for r in range(P)]
         return (torch.from_numpy(k[order].view(np.int64).copy()), torch.from_numpy(v[order].copy()), counts)
 
+    def validate(self, keys, vals, op) -> int:
+        """gpma_validate_batch: RESERVED (3) beats RANGE (2); global vertex range."""
+        k = keys.numpy().view(np.uint64)
+        src, dst = k >> np.uint64(32), k & np.uint64(0xFFFFFFFF)
+        if (dst == np.uint64(0xFFFFFFFF)).any():
+            return 3
+        if op == 0 and vals is not None and (vals.numpy().view(np.uint32) == np.uint32(0xFFFFFFFF)).any():
+            return 3
+        return 2 if ((src >= np.uint64(self.V)) | (dst >= np.uint64(self.V))).any() else 0
+
     def update(self, keys, vals, op):
         if op == 0:
             self.o.insert(keys.numpy(), vals.numpy())
@@ -126,6 +136,9 @@ class OracleShard:
         err = float(np.abs(nx - xv[lo:hi]).sum())
         xv[lo:hi] = nx
         return err
+
+    def pr_update_rows_dev(self, x, y_rows, damping, err_dev):
+        err_dev += self.pr_update_rows(x, y_rows, damping)
 
     def bfs_bits(self, levels, depth, bitmap):
         """gpma_bfs_bits: bit v of bitmap = (levels[v] == depth)."""

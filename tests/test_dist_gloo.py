@@ -64,6 +64,21 @@ def _worker(rank, world, port, mode, seed, fails):
             xo, _ = ref.pagerank(x=x, tol=0.0, max_iter=6)
             assert it == 6 and np.abs(xg.numpy() - xo).max() < 1e-12
             x = xo
+        # a bad key on ONE rank rejects the batch on every rank, nothing applied anywhere
+        before = shard.o.dump()
+        bad = torch.tensor([(V + 3) << 32 | 1] if rank == world - 1 else [], dtype=torch.int64)
+        from paper_journals_pvldb_shalht17_b200.gpma import GpmaError
+        try:
+            dg.insert(bad, torch.ones(bad.numel(), dtype=torch.int32))
+            raise AssertionError("the bad batch was accepted")
+        except GpmaError as e:
+            assert e.status == 2
+        after = shard.o.dump()
+        assert (before[0] == after[0]).all() and (before[1] == after[1]).all()
+        # tolerance mode: the same stopping iteration as the single store
+        xg, it = dg.pagerank(None, warm=False, tol=1e-3, max_iter=100)
+        xo, ito = ref.pagerank(tol=1e-3, max_iter=100)
+        assert it == ito and np.abs(xg.numpy() - xo).max() < 1e-12
         dist.destroy_process_group()
     except Exception as e:  # surface the failure to the parent
         import traceback
@@ -76,6 +91,16 @@ def test_two_rank_gloo_matches_single_store(mode, seed):
     ctx = mp.get_context("spawn")
     fails = ctx.Queue()
     mp.spawn(_worker, args=(2, _free_port(), mode, seed, fails), nprocs=2, join=True)
+    assert fails.empty()
+
+
+@pytest.mark.parametrize("world,seed", [(3, 7), (4, 8)])
+def test_ragged_shards_gloo_matches_single_store(world, seed):
+    """World size 3 and 4: V = 1024 splits into unequal row ranges (342/342/340, 256 x 4), batch
+    slices of unequal length; lazy deletes."""
+    ctx = mp.get_context("spawn")
+    fails = ctx.Queue()
+    mp.spawn(_worker, args=(world, _free_port(), O.LAZY, seed, fails), nprocs=world, join=True)
     assert fails.empty()
 
 
