@@ -29,19 +29,25 @@ def _store_pair(sw, V, mode=O.LAZY):
 
 
 def test_config2_full_size():
+    """configs[2] at full size, on a side stream exactly as bench.py drives it: slide 0 runs the
+    prefixes plainly, slide 1 captures them as CUDA graphs, slide 2 REPLAYS them (1M-key batches)."""
     cfg = CONFIGS[2]
     sw = config_stream(2, device=DEV)
     V = cfg.V
     g, o = _store_pair(sw, V)
     assert_same_layout(g, o, what="config2 create")
     x = None
-    for s in range(2):
+    st = torch.cuda.Stream()
+    for s in range(3):
         dk, ik, iv = sw.slide(s)
-        g.delete(dk.contiguous())
-        g.insert(ik.contiguous(), iv.contiguous())
+        with torch.cuda.stream(st):
+            g.gpma_update_batch(dk.contiguous(), None, 1, stream=st)
+            g.gpma_update_batch(ik.contiguous(), iv.contiguous(), 0, stream=st)
+        st.synchronize()
         o.delete(dk.cpu())
         o.insert(ik.cpu(), iv.cpu())
-        assert_same_layout(g, o, what=f"config2 slide {s}")
+        if s != 1:
+            assert_same_layout(g, o, what=f"config2 slide {s}")
     assert_same_csr(g, o, what="config2")
     root = bfs_root(sw, cfg.seed, 1)
     assert np.array_equal(gpu_bfs(g, root), o.bfs(root))
@@ -104,3 +110,48 @@ def test_config3_resize_stress_scaled():
     assert caps[-1] < max(caps), "no halving happened"
     assert g.gpma_stats()["resizes"] == o.stats()["resizes"]
     assert_same_csr(g, o, what="config3-scaled")
+
+
+def _resize_pair(V, cap0, E0, seed, mode):
+    """A configs[3]-shaped store (V = 2^24, uniform edges) created at capacity cap0 (override) on
+    both sides, the edges' stream returned for the batches that follow."""
+    from paper_journals_pvldb_shalht17_b200 import Gpma
+    pool = make_stream("uniform", V, E0 + (1 << 21), seed, device=DEV)
+    vals = edge_values(pool, seed)
+    g = Gpma.gpma_create(V, pool[:E0].contiguous(), vals[:E0].contiguous(), delete_mode=mode, initial_capacity=cap0)
+    o = O.Oracle(V, pool[:E0].cpu(), vals[:E0].cpu(), delete_mode=mode, capacity=cap0)
+    return g, o, pool, vals
+
+
+def test_config3_full_size_doubling():
+    """configs[3] at full size (V = 2^24): a store at capacity 2^26 holding just under the root
+    bound max_h (R5) takes one hot 2^20-edge insert batch whose climb reaches the root, which
+    doubles to 2^27 (Alg. 4 l.16-17, R14) -- the whole 2^27-slot layout against the oracle."""
+    V, cap0 = 1 << 24, 1 << 26
+    mx = O.thresholds(16, 22)[1][22]
+    E0 = mx - V - (1 << 18)
+    g, o, pool, vals = _resize_pair(V, cap0, E0, CONFIGS[3].seed + 11, 0)
+    # a hot batch (NEXT-4 shape): 2^20 new edges from 64 consecutive rows, so every window that
+    # holds them is over its bound up to the root (an even one would be absorbed at the leaves)
+    i = torch.arange(1 << 20, device=DEV)
+    ik = (((1000 + i // (1 << 14)) << 32) | ((i % (1 << 14)) * 1021 % V)).contiguous()
+    iv = (i % 1000).to(torch.int32).contiguous()
+    g.insert(ik, iv)
+    o.insert(ik.cpu(), iv.cpu())
+    assert o.capacity == 1 << 27 and o.stats()["resizes"] == 1
+    assert_same_layout(g, o, what="config3 doubling 2^26 -> 2^27")
+    assert g.gpma_stats()["resizes"] == 1
+
+
+def test_config3_full_size_halving():
+    """configs[3] at full size, strict deletes: a store at capacity 2^28 far below the root's
+    lower bound (V guards + 2^22 edges) -- every deletion climbs to the root, which halves while
+    N < min_h and the half can hold N (R14): 2^28 -> 2^25 in one batch, compared slot by slot."""
+    V, cap0, E0 = 1 << 24, 1 << 28, 1 << 22
+    g, o, pool, vals = _resize_pair(V, cap0, E0, CONFIGS[3].seed + 12, 1)
+    dk = pool[: 1 << 20].contiguous()
+    g.delete(dk)
+    o.delete(dk.cpu())
+    assert o.capacity < cap0 and o.stats()["resizes"] >= 1
+    assert_same_layout(g, o, what=f"config3 halving 2^28 -> {o.capacity}")
+    assert g.gpma_stats()["capacity"] == o.capacity
