@@ -553,32 +553,21 @@ __global__ void __launch_bounds__(256) k_ins_leaf_t(const uint64_t *__restrict__
     news += nnew;
     if (ok) {
       const uint64_t h_old = K[0];
-      // drop the remaining tombstones: left-pack the live entries (static select network)
-      if (live != ((1u << n) - 1u)) {
-        uint64_t K2[L];
-        uint32_t V2[L];
+      if (live != ((1u << n) - 1u)) {                   // drop the tombstones (highest first: the
+        uint32_t dead = occ & ~live;                    // lower positions stay valid), left-packing
+        while (dead) {
+          const int pd = 31 - __clz(dead);
 #pragma unroll
-        for (int q = 0; q < L; ++q) {
-          K2[q] = KEY_NONE;
-          V2[q] = 0;
-        }
-#pragma unroll
-        for (int p = 0; p < L; ++p) {
-          const uint32_t r = __popc(live & ((1u << p) - 1u));      // rank of slot p among the live
-#pragma unroll
-          for (int q = 0; q <= p; ++q)
-            if (((live >> p) & 1u) && r == (uint32_t)q) {
-              K2[q] = K[p];
-              V2[q] = Vv[p];
+          for (int p = 0; p < L - 1; ++p)
+            if (p >= pd) {
+              K[p] = K[p + 1];
+              Vv[p] = Vv[p + 1];
             }
-        }
-#pragma unroll
-        for (int q = 0; q < L; ++q) {
-          K[q] = K2[q];
-          Vv[q] = V2[q];
+          K[L - 1] = KEY_NONE;
+          Vv[L - 1] = 0;
+          dead &= ~(1u << pd);
         }
       }
-      // merge the new keys (sorted) into the live prefix, one static shift each
       uint32_t N = n;
       for (uint32_t j = j0; j < j1; ++j) {
         const uint64_t uk = sk[j];
@@ -804,28 +793,19 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
     news += nnew;
     if (ok) {
       const uint64_t h_old = K[0];
-      if (live != ((1u << n) - 1u)) {                   // drop the tombstones: left-pack the live
-        uint64_t K2[L];
-        uint32_t V2[L];
+      if (live != ((1u << n) - 1u)) {                   // drop the tombstones (highest first: the
+        uint32_t dead = occ & ~live;                    // lower positions stay valid), left-packing
+        while (dead) {
+          const int pd = 31 - __clz(dead);
 #pragma unroll
-        for (int q = 0; q < L; ++q) {
-          K2[q] = KEY_NONE;
-          V2[q] = 0;
-        }
-#pragma unroll
-        for (int p = 0; p < L; ++p) {
-          const uint32_t r = __popc(live & ((1u << p) - 1u));
-#pragma unroll
-          for (int q = 0; q <= p; ++q)
-            if (((live >> p) & 1u) && r == (uint32_t)q) {
-              K2[q] = K[p];
-              V2[q] = Vv[p];
+          for (int p = 0; p < L - 1; ++p)
+            if (p >= pd) {
+              K[p] = K[p + 1];
+              Vv[p] = Vv[p + 1];
             }
-        }
-#pragma unroll
-        for (int q = 0; q < L; ++q) {
-          K[q] = K2[q];
-          Vv[q] = V2[q];
+          K[L - 1] = KEY_NONE;
+          Vv[L - 1] = 0;
+          dead &= ~(1u << pd);
         }
       }
       uint32_t N = n;
@@ -942,6 +922,167 @@ __global__ void k_pend_permute(const uint32_t *__restrict__ perm, uint64_t p, co
     const uint32_t q = perm[j];
     pv[j] = pv_in[q];
     pt[j] = pt_in[q];
+  }
+}
+
+// ---- R-way interleaved locate (memory-level parallelism): the random loads of R independent
+// keys -- row offsets, head probes, the first 8 slots of the target leaf -- are issued together,
+// so a thread keeps R dependent chains in flight instead of one (the kernels below are bound by
+// DRAM latency at full occupancy: one chain per thread left DRAM at ~43 % of its bandwidth).
+template <int R>
+__device__ __forceinline__ void locate_leaf_rows_r(const uint64_t *__restrict__ head, uint32_t nleaves,
+                                                   const uint64_t *__restrict__ ro, uint32_t rb, uint32_t L,
+                                                   const uint64_t (&k)[R], const bool (&v)[R], uint32_t (&t)[R]) {
+  uint32_t lo[R], hi[R], a[R];
+  if (!ro) {
+#pragma unroll
+    for (int q = 0; q < R; ++q) t[q] = v[q] ? locate_leaf(head, nleaves, k[q]) : 0u;
+    return;
+  }
+  ulonglong2 r[R];
+#pragma unroll
+  for (int q = 0; q < R; ++q) {
+    const uint32_t u = (uint32_t)(k[q] >> 32) - rb;
+    r[q] = v[q] ? make_ulonglong2(__ldg(ro + u), __ldg(ro + u + 1)) : make_ulonglong2(0, 0);
+  }
+#pragma unroll
+  for (int q = 0; q < R; ++q) {
+    a[q] = (uint32_t)leaf_div(r[q].x, L);
+    lo[q] = a[q];
+    hi[q] = v[q] ? min((uint32_t)leaf_div(r[q].y, L) + 1, nleaves) : a[q];
+  }
+  bool any = true;
+  while (any) {
+    uint64_t hv[R];
+    uint32_t mid[R];
+#pragma unroll
+    for (int q = 0; q < R; ++q) {
+      mid[q] = (lo[q] + hi[q]) >> 1;
+      hv[q] = lo[q] < hi[q] ? __ldg(head + mid[q]) : 0ull;
+    }
+    any = false;
+#pragma unroll
+    for (int q = 0; q < R; ++q)
+      if (lo[q] < hi[q]) {
+        if (hv[q] <= k[q]) lo[q] = mid[q] + 1;
+        else hi[q] = mid[q];
+        any |= lo[q] < hi[q];
+      }
+  }
+#pragma unroll
+  for (int q = 0; q < R; ++q) t[q] = lo[q] > a[q] ? lo[q] - 1 : a[q];
+}
+
+// slot of k[q] in its leaf t[q] (or -1) for R keys: the leaves' slots fetched 8 at a time, the
+// R leaves of a round together (the occupied prefix is sorted, KEY_NONE > every key)
+template <int R>
+__device__ __forceinline__ void find_in_leaf_r(const uint64_t *__restrict__ key, uint32_t L, const uint64_t (&k)[R],
+                                               const bool (&v)[R], const uint32_t (&t)[R], int (&pos)[R]) {
+  bool more[R];
+#pragma unroll
+  for (int q = 0; q < R; ++q) {
+    pos[q] = -1;
+    more[q] = v[q];
+  }
+  for (uint32_t p0 = 0; p0 < L; p0 += 8) {
+    bool any = false;
+#pragma unroll
+    for (int q = 0; q < R; ++q) any |= more[q];
+    if (!any) break;
+    ulonglong2 a[R][4];
+#pragma unroll
+    for (int q = 0; q < R; ++q)
+#pragma unroll
+      for (int j = 0; j < 4; ++j)
+        a[q][j] = more[q] && p0 + 2 * j < L
+                      ? __ldg(reinterpret_cast<const ulonglong2 *>(key + (uint64_t)t[q] * L + p0 + 2 * j))
+                      : make_ulonglong2(KEY_NONE, KEY_NONE);
+#pragma unroll
+    for (int q = 0; q < R; ++q) {
+#pragma unroll
+      for (int j = 0; j < 4; ++j) {
+        if (!more[q]) break;
+        if (a[q][j].x == k[q]) { pos[q] = (int)(p0 + 2 * j); more[q] = false; }
+        else if (a[q][j].x > k[q]) more[q] = false;
+        else if (a[q][j].y == k[q]) { pos[q] = (int)(p0 + 2 * j + 1); more[q] = false; }
+        else if (a[q][j].y > k[q]) more[q] = false;
+      }
+    }
+  }
+}
+
+// Lazy deletion (R12) in arrival order, R keys per thread interleaved.  Duplicates
+// race on the same slot; the CAS on the value lets exactly one account the deletion.
+template <int LD_R>
+__global__ void __launch_bounds__(256) k_lazy_delete_r(const uint64_t *__restrict__ keys, uint64_t n,
+                                                       const uint64_t *__restrict__ key, uint32_t *val,
+                                                       uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
+                                                       uint32_t nleaves, uint32_t L, uint32_t *__restrict__ tmask,
+                                                       uint32_t *__restrict__ deg, uint32_t rb, const Ctrl *c,
+                                                       const uint64_t *__restrict__ ro) {
+  if (c->err) return;
+  const uint64_t nthr = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i0 < n; i0 += nthr * LD_R) {
+    uint64_t k[LD_R];
+    bool v[LD_R];
+#pragma unroll
+    for (int q = 0; q < LD_R; ++q) {
+      const uint64_t i = i0 + (uint64_t)q * nthr;
+      v[q] = i < n;
+      k[q] = v[q] ? keys[i] : 0ull;
+    }
+    uint32_t t[LD_R];
+    locate_leaf_rows_r<LD_R>(head, nleaves, ro, rb, L, k, v, t);
+    int p[LD_R];
+    find_in_leaf_r<LD_R>(key, L, k, v, t, p);
+    uint32_t old[LD_R];
+#pragma unroll
+    for (int q = 0; q < LD_R; ++q) old[q] = p[q] >= 0 ? val[(uint64_t)t[q] * L + p[q]] : VAL_TOMB;
+#pragma unroll
+    for (int q = 0; q < LD_R; ++q) {
+      const uint64_t s = (uint64_t)t[q] * L + (p[q] >= 0 ? p[q] : 0);
+      while (old[q] != VAL_TOMB) {
+        const uint32_t seen = atomicCAS(&val[s], old[q], VAL_TOMB);
+        if (seen == old[q]) {
+          atomicSub(&cnt[t[q]], 1u);
+          atomicOr(&tmask[t[q]], 1u << p[q]);
+          atomicSub(&deg[(uint32_t)(k[q] >> 32) - rb], 1u);
+          break;
+        }
+        old[q] = seen;
+      }
+    }
+  }
+}
+
+// Target leaf of every update of the unsorted batch, R keys per thread interleaved
+template <int LD_R>
+__global__ void __launch_bounds__(256) k_locate_u_r(const uint64_t *__restrict__ ik, uint64_t n,
+                                                    const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
+                                                    uint32_t rb, const uint64_t *__restrict__ ro,
+                                                    uint64_t *__restrict__ tk, uint32_t *__restrict__ tix,
+                                                    const Ctrl *c) {
+  if (c->err) return;
+  const uint64_t nthr = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i0 < n; i0 += nthr * LD_R) {
+    uint64_t k[LD_R];
+    bool v[LD_R];
+#pragma unroll
+    for (int q = 0; q < LD_R; ++q) {
+      const uint64_t i = i0 + (uint64_t)q * nthr;
+      v[q] = i < n;
+      k[q] = v[q] ? ik[i] : 0ull;
+    }
+    uint32_t t[LD_R];
+    locate_leaf_rows_r<LD_R>(head, nleaves, ro, rb, L, k, v, t);
+#pragma unroll
+    for (int q = 0; q < LD_R; ++q) {
+      const uint64_t i = i0 + (uint64_t)q * nthr;
+      if (v[q]) {
+        tk[i] = t[q];
+        tix[i] = (uint32_t)i;
+      }
+    }
   }
 }
 
@@ -2485,6 +2626,12 @@ static int prefix_path(gpma *g, int op) {
   return PATH_GENERIC;
 }
 
+// GPMA_ILP = keys per thread of the random-probe kernels (lazy delete, locate): 1, 2 or 4
+static int ilp_r() {
+  const char *e = getenv("GPMA_ILP");
+  return e ? atoi(e) : 2;
+}
+
 static int leaf_shifts(uint64_t nleaves, int *sh) {
   const uint32_t bits = nleaves <= 1 ? 1 : ilog2(nleaves - 1) + 1;
   int n = 0;
@@ -2510,8 +2657,16 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
   const uint64_t *ro = g->rows_indexed ? g->row_offset : nullptr;
   const int path = prefix_path(g, op);
   if (path == PATH_LAZY_UNSORTED) {
-    GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
-              tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
+    const int R = ilp_r();
+    if (R >= 4)
+      GP_LAUNCH(g, k_lazy_delete_r<4>, grid_for((n + 3) / 4), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head,
+                (uint32_t)nl, g->L, tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
+    else if (R == 2)
+      GP_LAUNCH(g, k_lazy_delete_r<2>, grid_for((n + 1) / 2), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head,
+                (uint32_t)nl, g->L, tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
+    else
+      GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
+                tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
     GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
     return GPMA_OK;
   }
@@ -2527,7 +2682,15 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
     GP_CHECK(g, ensure(g, g->b_sv[1], n * 4, s));
     uint64_t *tk0 = (uint64_t *)g->b_sk[0].p, *tk1 = (uint64_t *)g->b_sk[1].p;
     uint32_t *tx0 = (uint32_t *)g->b_sv[0].p, *tx1 = (uint32_t *)g->b_sv[1].p;
-    GP_LAUNCH(g, k_locate_u, grid_for(n), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0, tx0, g->ctrl_d);
+    const int R = ilp_r();
+    if (R >= 4)
+      GP_LAUNCH(g, k_locate_u_r<4>, grid_for((n + 3) / 4), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0,
+                tx0, g->ctrl_d);
+    else if (R == 2)
+      GP_LAUNCH(g, k_locate_u_r<2>, grid_for((n + 1) / 2), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0,
+                tx0, g->ctrl_d);
+    else
+      GP_LAUNCH(g, k_locate_u, grid_for(n), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0, tx0, g->ctrl_d);
     int sh[8], which = 0;
     const int ns = leaf_shifts(nl, sh);
     GP_CHECK(g, radix_sort_pairs(g, tk0, tx0, tk1, tx1, n, sh, ns, s, &which));
