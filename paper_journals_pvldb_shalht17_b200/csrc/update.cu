@@ -751,19 +751,15 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
       }
     }
     __syncwarp();
-    uint64_t K[L];
-    uint32_t Vv[L];
-#pragma unroll
-    for (int p = 0; p < L; ++p) {
-      K[p] = have ? mk[lane * KS + p] : KEY_NONE;
-      Vv[p] = have ? mv[lane * KS + p] : 0u;
+    // the thread's leaf is its row of shared memory: dynamic indexing is free there, so the
+    // merge is a few moves per update instead of static select networks over registers
+    uint64_t *const rk = mk + lane * KS;
+    uint32_t *const rv = mv + lane * KS;
+    uint32_t nocc = 0, tomb = 0;
+    if (have) {
+      for (; nocc < (uint32_t)L && rk[nocc] != KEY_NONE; ++nocc) tomb |= (rv[nocc] == VAL_TOMB ? 1u : 0u) << nocc;
     }
-    uint32_t occ = 0, tomb = 0;
-#pragma unroll
-    for (int p = 0; p < L; ++p) {
-      occ |= (K[p] != KEY_NONE ? 1u : 0u) << p;
-      tomb |= (K[p] != KEY_NONE && Vv[p] == VAL_TOMB ? 1u : 0u) << p;
-    }
+    const uint64_t h_old = have ? rk[0] : KEY_NONE;
     uint32_t hitm = 0, revm = 0, nnew = 0;
     for (uint32_t j = j0; j < j1; ++j) {
       const uint32_t i = tix[j];
@@ -773,13 +769,16 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
       uint32_t h = 0;
       if (last) {
         ++effs;
-        const uint32_t uv = iv[i];
-#pragma unroll
-        for (int p = 0; p < L; ++p)
-          if (K[p] == uk) {
-            h = 1u << p;
-            Vv[p] = uv;
-          }
+        uint32_t lo = 0, hi = nocc;                      // the occupied prefix is sorted
+        while (lo < hi) {
+          const uint32_t mid = (lo + hi) >> 1;
+          if (rk[mid] < uk) lo = mid + 1;
+          else hi = mid;
+        }
+        if (lo < nocc && rk[lo] == uk) {                 // overwrite (R11) / revive (R12)
+          h = 1u << lo;
+          rv[lo] = iv[i];
+        }
         hitm |= h;
         revm |= h & tomb;
         nnew += h ? 0u : 1u;
@@ -787,84 +786,57 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
       }
       keep[j] = (last && !h) ? 1u : 0u;
     }
-    const uint32_t live = occ & ~(tomb & ~revm);
-    const uint32_t n = __popc(live);
+    const uint32_t dead = tomb & ~revm;
+    const uint32_t n = nocc - __popc(dead);
     const bool ok = have && nnew > 0 && nnew <= bound && n + nnew <= bound;
     news += nnew;
     if (ok) {
-      const uint64_t h_old = K[0];
-      if (live != ((1u << n) - 1u)) {                   // drop the tombstones (highest first: the
-        uint32_t dead = occ & ~live;                    // lower positions stay valid), left-packing
-        while (dead) {
-          const int pd = 31 - __clz(dead);
-#pragma unroll
-          for (int p = 0; p < L - 1; ++p)
-            if (p >= pd) {
-              K[p] = K[p + 1];
-              Vv[p] = Vv[p + 1];
-            }
-          K[L - 1] = KEY_NONE;
-          Vv[L - 1] = 0;
-          dead &= ~(1u << pd);
-        }
-      }
       uint32_t N = n;
-      for (uint32_t j = j0; j < j1; ++j) {
+      if (dead) {                                        // drop the tombstones: left-pack the live
+        uint32_t w2 = 0;
+        for (uint32_t p = 0; p < nocc; ++p)
+          if (!((dead >> p) & 1u)) {
+            rk[w2] = rk[p];
+            rv[w2] = rv[p];
+            ++w2;
+          }
+      }
+      for (uint32_t j = j0; j < j1; ++j) {               // the new keys at their key rank
         if (!keep[j]) continue;
         keep[j] = 0u;
         const uint32_t i = tix[j];
         const uint64_t uk = ik[i];
-        const uint32_t uv = iv[i];
-        uint32_t pos = 0;
-#pragma unroll
-        for (int p = 0; p < L; ++p) pos += (p < (int)N) && K[p] < uk;
-#pragma unroll
-        for (int p = L - 1; p > 0; --p)
-          if ((uint32_t)p > pos) {
-            K[p] = K[p - 1];
-            Vv[p] = Vv[p - 1];
-          }
-#pragma unroll
-        for (int p = 0; p < L; ++p)
-          if ((uint32_t)p == pos) {
-            K[p] = uk;
-            Vv[p] = uv;
-          }
+        uint32_t pos = N;
+        while (pos > 0 && rk[pos - 1] > uk) {
+          rk[pos] = rk[pos - 1];
+          rv[pos] = rv[pos - 1];
+          --pos;
+        }
+        rk[pos] = uk;
+        rv[pos] = iv[i];
         ++N;
       }
-#pragma unroll
-      for (int p = 0; p < L; ++p)
-        if ((uint32_t)p >= N) {
-          K[p] = KEY_NONE;
-          Vv[p] = 0;
-        }
-#pragma unroll
-      for (int p = 0; p < L; ++p) {
-        mk[lane * KS + p] = K[p];
-        mv[lane * KS + p] = Vv[p];
-        if (is_guard_key(K[p])) row_offset[(K[p] >> 32) - rb + 1] = lb + p;   // R8: guards that moved
+      for (uint32_t p = N; p < nocc; ++p) {
+        rk[p] = KEY_NONE;
+        rv[p] = 0;
       }
+      for (uint32_t p = 0; p < N; ++p)
+        if (is_guard_key(rk[p])) row_offset[(rk[p] >> 32) - rb + 1] = lb + p;   // R8: guards that moved
       cnt[t] = N;
       if (tomb) tmask[t] = 0u;                          // (no tombstone in the leaf: already 0)
-      if (K[0] != h_old) {
-        head[t] = K[0];
+      if (rk[0] != h_old) {
+        head[t] = rk[0];
         if (t > 0 && key[lb - L] == KEY_NONE) {          // empty leaves to the left carry this head
           const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
           dirty[d] = make_uint2(t, 1u);
         }
       }
       ++accepted;
-    } else if (have) {
-      if (hitm) {
-#pragma unroll
-        for (int p = 0; p < L; ++p)
-          if ((hitm >> p) & 1u) val[lb + p] = Vv[p];
-      }
-      if (revm) {
-        cnt[t] += __popc(revm);
-        tmask[t] &= ~revm;
-      }
+    } else if (have && revm) {
+      cnt[t] += __popc(revm);
+      tmask[t] &= ~revm;
     }
+    const bool vdirty = ok || hitm;                      // the values go back for hits too
     __syncwarp();
     // cooperative store of the accepted (rewritten) leaves
 #pragma unroll
@@ -879,7 +851,7 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
     for (int it = 0; it < 32 / VQ; ++it) {
       const int q = it * VQ + lane / VL, cc = lane % VL;
       const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
-      const bool oq = __shfl_sync(0xffffffffu, ok, q);
+      const bool oq = __shfl_sync(0xffffffffu, vdirty, q);
       if (oq)
         *reinterpret_cast<uint4 *>(val + lq + 4 * cc) =
             make_uint4(mv[q * KS + 4 * cc], mv[q * KS + 4 * cc + 1], mv[q * KS + 4 * cc + 2], mv[q * KS + 4 * cc + 3]);
