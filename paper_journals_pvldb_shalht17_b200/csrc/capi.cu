@@ -119,9 +119,11 @@ gpma *new_handle(uint32_t V) {
   if (!g) return nullptr;
   g->V = V;
   if (cudaMalloc((void **)&g->ctrl_d, sizeof(gp::Ctrl)) != cudaSuccess ||
-      cudaMallocHost((void **)&g->ctrl_h, sizeof(gp::Ctrl)) != cudaSuccess) {
+      cudaMallocHost((void **)&g->ctrl_h, sizeof(gp::Ctrl)) != cudaSuccess ||
+      cudaMallocHost(&g->pin, 256) != cudaSuccess) {
     cudaGetLastError();
     if (g->ctrl_d) cudaFree(g->ctrl_d);
+    if (g->ctrl_h) cudaFreeHost(g->ctrl_h);
     delete g;
     return nullptr;
   }
@@ -169,6 +171,7 @@ void free_handle(gpma *g) {
   for (cudaEvent_t e : g->ev_pool) cudaEventDestroy(e);
   if (g->ctrl_d) cudaFree(g->ctrl_d);
   if (g->ctrl_h) cudaFreeHost(g->ctrl_h);
+  if (g->pin) cudaFreeHost(g->pin);
   for (gp::Scratch &x : g->an) {
     if (x.ctrl_d) cudaFree(x.ctrl_d);
     if (x.ctrl_h) cudaFreeHost(x.ctrl_h);

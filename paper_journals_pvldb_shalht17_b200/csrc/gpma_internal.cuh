@@ -121,6 +121,7 @@ struct gpma {
   gp::DevBuf b_lpre, b_wk, b_wv, b_dirty, b_scan, b_hist, b_stage[4], b_misc, b_misc2, b_misc3;
   gp::Ctrl *ctrl_d = nullptr;
   gp::Ctrl *ctrl_h = nullptr;     // pinned mirror
+  void *pin = nullptr;            // 256 B of pinned host scratch (read-backs of small device state)
   gp::Scratch an[gp::AN_N];       // analytics (read-only on the store)
 
   // device memory (gpma_config.alloc / free / alloc_ctx; NULL = the library's pool)

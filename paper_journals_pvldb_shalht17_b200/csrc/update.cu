@@ -15,6 +15,8 @@
 // list (gather -> scatter), so no kernel ever reads a slot another CTA writes.
 #include <cuda_runtime.h>
 
+#include <cooperative_groups.h>
+
 #include <algorithm>
 
 #include "gpma_internal.cuh"
@@ -1759,6 +1761,307 @@ __global__ void k_lvl_summary(Lvl a, Ctrl *c) {
   c->sum2 = a.kpos[a.p];
 }
 
+// ---- device-resident level loop (Alg. 4 l.4-15 above the leaves) ----------------------------
+// One cooperative kernel runs levels 1, 2, ... on the device while the pending list is small
+// (<= CL_MAXP) and the windows fit a CTA's shared memory (<= CL_MAXS slots, TryInsert+ at
+// block scale): per level, CTA 0 forms the segments (UniqueSegments = RLE + scan,
+// l.18-21), every warp counts a window and tests it (CountSegment + density, l.23-25), every
+// CTA merges and re-dispatches accepted windows in shared memory (l.26-27, R7), CTA 0 promotes
+// the rest (l.12-15) -- grid-wide barriers between the phases instead of a host round trip per
+// level.  It stops at the first level it cannot take; the host continues from there (larger
+// windows, the root resize).
+constexpr int CL_T = 512, CL_I = 16;
+constexpr uint32_t CL_MAXP = CL_T * CL_I;            // 8192 pending updates
+constexpr uint32_t CL_MAXS = 4096;                   // slots of the largest window (48 KiB of keys + values)
+
+struct CoopState {
+  uint64_t p;                  // pending entering the level
+  uint32_t cur, lvl, done, q;  // pending buffer, level, stop flag, windows of the level
+  uint64_t windows, slots;     // rewritten by this kernel
+  uint32_t top;                // highest level that ran
+};
+
+struct CoopArgs {
+  uint64_t *pk[2];
+  uint32_t *pv[2], *pt[2];
+  uint32_t *hf, *widx, *wfirst, *acc, *keep, *kpos;
+  uint64_t *nw;
+  uint64_t *key;
+  uint32_t *val, *cnt, *tmask;
+  uint64_t *row_offset;
+  uint2 *dirty;
+  uint64_t nleaves;
+  uint32_t L, h, rb;
+  int op;
+  uint64_t tmin[48], tmax[48];
+  CoopState *st;
+  Ctrl *c;
+};
+
+// exclusive scan of CL_I consecutive items per thread over the CTA; returns the total
+__device__ __forceinline__ uint64_t cl_scan(uint64_t (&v)[CL_I], uint64_t *wsum) {
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  uint64_t ex[CL_I];
+  uint64_t t = 0;
+#pragma unroll
+  for (int i = 0; i < CL_I; ++i) {
+    ex[i] = t;
+    t += v[i];
+  }
+  uint64_t x = t;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint64_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if (lane >= o) x += y;
+  }
+  if (lane == 31) wsum[warp] = x;
+  __syncthreads();
+  if (warp == 0) {
+    uint64_t w = lane < CL_T / 32 ? wsum[lane] : 0;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint64_t y = __shfl_up_sync(0xffffffffu, w, o);
+      if (lane >= o) w += y;
+    }
+    if (lane < CL_T / 32) wsum[lane] = w;
+  }
+  __syncthreads();
+  const uint64_t base = (warp ? wsum[warp - 1] : 0) + x - t;
+  const uint64_t total = wsum[CL_T / 32 - 1];
+  __syncthreads();
+#pragma unroll
+  for (int i = 0; i < CL_I; ++i) v[i] = base + ex[i];
+  return total;
+}
+
+// CTA 0: the segments of level S.lvl over the pending list S.cur (hf, widx, wfirst, q)
+__device__ void cl_segments(const CoopArgs &a, CoopState &S, uint64_t *wsum) {
+  const uint64_t p = S.p;
+  const uint32_t lvl = S.lvl;
+  const uint32_t *pt = a.pt[S.cur];
+  const uint64_t j0 = (uint64_t)threadIdx.x * CL_I;
+  uint64_t f[CL_I], e[CL_I];
+#pragma unroll
+  for (int i = 0; i < CL_I; ++i) {
+    const uint64_t j = j0 + i;
+    f[i] = (j < p && (j == 0 || (pt[j] >> lvl) != (pt[j - 1] >> lvl))) ? 1u : 0u;
+    if (j < p) a.hf[j] = (uint32_t)f[i];
+    e[i] = f[i];
+  }
+  const uint64_t q = cl_scan(e, wsum);
+#pragma unroll
+  for (int i = 0; i < CL_I; ++i) {
+    const uint64_t j = j0 + i;
+    if (j < p) {
+      a.widx[j] = (uint32_t)e[i];
+      if (f[i]) a.wfirst[e[i]] = (uint32_t)j;
+    }
+  }
+  if (threadIdx.x == 0) {
+    a.widx[p] = (uint32_t)q;
+    a.wfirst[q] = (uint32_t)p;
+    S.q = (uint32_t)q;
+  }
+}
+
+// CTA 0: promote the rejected updates of the level to the next buffer (l.12-15), next level
+__device__ void cl_promote(const CoopArgs &a, CoopState &S, uint64_t *wsum) {
+  const uint64_t p = S.p;
+  const uint32_t cur = S.cur;
+  const uint64_t j0 = (uint64_t)threadIdx.x * CL_I;
+  uint64_t k[CL_I], kk[CL_I];
+#pragma unroll
+  for (int i = 0; i < CL_I; ++i) {
+    const uint64_t j = j0 + i;
+    k[i] = 0;
+    if (j < p) {
+      const uint32_t w = a.widx[j] + a.hf[j] - 1;
+      k[i] = a.acc[w] ? 0u : 1u;
+    }
+    kk[i] = k[i];
+  }
+  const uint64_t pn = cl_scan(kk, wsum);
+#pragma unroll
+  for (int i = 0; i < CL_I; ++i) {
+    const uint64_t j = j0 + i;
+    if (j < p && k[i]) {
+      a.pk[cur ^ 1][kk[i]] = a.pk[cur][j];
+      a.pv[cur ^ 1][kk[i]] = a.pv[cur][j];
+      a.pt[cur ^ 1][kk[i]] = a.pt[cur][j];
+    }
+  }
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    S.top = S.lvl;
+    S.p = pn;
+    if (pn) S.cur = cur ^ 1;
+    S.lvl += 1;
+    S.done = (pn == 0 || S.lvl > a.h || ((uint64_t)a.L << S.lvl) > CL_MAXS) ? 1u : 0u;
+  }
+  __syncthreads();
+  __threadfence_block();
+}
+
+// one accepted window merged and re-dispatched in shared memory (CTA-wide, Alg. 4 l.26-27)
+__device__ void cl_merge_window(const CoopArgs &a, const CoopState &S, uint32_t w, uint64_t *mk, uint32_t *mv,
+                                uint32_t *lpre) {
+  const uint32_t lvl = S.lvl, L = a.L;
+  const uint64_t *pk = a.pk[S.cur];
+  const uint32_t *pv = a.pv[S.cur], *pt = a.pt[S.cur];
+  const uint32_t Lc = 1u << lvl, ws = L << lvl;
+  const uint64_t leaf0 = ((uint64_t)(pt[a.wfirst[w]] >> lvl)) << lvl;
+  const uint64_t N = a.nw[w];
+  const uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint32_t leafmask = (L == 32 ? 0xffffffffu : ((1u << L) - 1u) << (lane & ~(L - 1)));
+  // live entries before each leaf of the window (Lc <= 256)
+  if (threadIdx.x < 32) {
+    uint32_t carry = 0;
+    for (uint32_t l0 = 0; l0 < Lc; l0 += 32) {
+      const uint32_t l = l0 + lane;
+      const uint32_t c0 = l < Lc ? a.cnt[leaf0 + l] : 0u;
+      uint32_t x = c0;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+        if (lane >= o) x += y;
+      }
+      if (l < Lc) lpre[l] = carry + x - c0;
+      carry += __shfl_sync(0xffffffffu, x, 31);
+    }
+    if (lane == 0) lpre[Lc] = carry;
+  }
+  __syncthreads();
+  for (uint32_t o0 = 0; o0 < ws; o0 += CL_T) {           // gather the live entries (whole warps)
+    const uint32_t off = o0 + threadIdx.x;
+    const bool in = off < ws;
+    uint64_t k = KEY_NONE;
+    uint32_t v = 0;
+    if (in) {
+      k = a.key[leaf0 * L + off];
+      v = a.val[leaf0 * L + off];
+    }
+    const bool live = in && k != KEY_NONE && v != VAL_TOMB;
+    const uint32_t bal = __ballot_sync(0xffffffffu, live);
+    if (live) {
+      const uint64_t rl = __popc(bal & leafmask & lt) + lpre[leaf_div(off, L)];
+      const uint64_t cc = lower_bound_u64(pk, ub, ue, k) - ub;
+      bool drop = false;
+      uint64_t r;
+      if (a.op == GPMA_INSERT) {
+        r = rl + cc;
+      } else {
+        drop = (ub + cc < ue) && pk[ub + cc] == k;
+        r = rl - cc;
+      }
+      if (!drop) {
+        mk[r] = k;
+        mv[r] = v;
+      }
+    }
+  }
+  if (a.op == GPMA_INSERT) {                             // place the window's insertions
+    for (uint64_t j = ub + threadIdx.x; j < ue; j += CL_T) {
+      const uint64_t k = pk[j];
+      const uint32_t t = pt[j];
+      uint64_t rl = lpre[t - leaf0];
+      const uint64_t base = (uint64_t)t * L;
+      for (uint32_t q = 0; q < L; ++q) {
+        const uint64_t x = a.key[base + q];
+        if (x == KEY_NONE || x > k) break;
+        if (a.val[base + q] != VAL_TOMB) ++rl;
+      }
+      const uint64_t r = (j - ub) + rl;
+      mk[r] = k;
+      mv[r] = pv[j];
+    }
+  }
+  __syncthreads();                                       // every read of the window is done
+  for (uint32_t off = threadIdx.x; off < ws; off += CL_T) {   // re-dispatch evenly (R7)
+    const uint64_t l = leaf_div(off, L), q = leaf_mod(off, L);
+    const uint64_t lo = l * N / Lc, hi = (l + 1) * N / Lc;
+    const uint64_t sl = leaf0 * L + off;
+    if (q < hi - lo) {
+      const uint64_t k = mk[lo + q];
+      a.key[sl] = k;
+      a.val[sl] = mv[lo + q];
+      if (is_guard_key(k)) a.row_offset[(k >> 32) - a.rb + 1] = sl;
+    } else {
+      a.key[sl] = KEY_NONE;
+      a.val[sl] = 0;
+    }
+    if (q == 0) {
+      a.cnt[leaf0 + l] = (uint32_t)(hi - lo);
+      a.tmask[leaf0 + l] = 0u;                           // tombstones are dropped by a rewrite
+      uint32_t gc = 0;
+      for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(mk[e]);
+      a.tmask[a.nleaves + leaf0 + l] = gc;               // guards per leaf (third section)
+    }
+  }
+  if (threadIdx.x == 0) {
+    const uint64_t d = atomicAdd((unsigned long long *)&a.c->ndirty, 1ull);
+    a.dirty[d] = make_uint2((uint32_t)leaf0, Lc);
+  }
+  __syncthreads();                                       // the smem list is reused by the next window
+}
+
+__global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
+  extern __shared__ __align__(16) unsigned char cl_smem[];
+  uint64_t *mk = reinterpret_cast<uint64_t *>(cl_smem);
+  uint32_t *mv = reinterpret_cast<uint32_t *>(mk + CL_MAXS);
+  uint32_t *lpre = mv + CL_MAXS;                         // [257]
+  __shared__ uint64_t wsum[CL_T / 32];
+  cooperative_groups::grid_group grid = cooperative_groups::this_grid();
+  CoopState &S = *a.st;
+  if (blockIdx.x == 0) cl_segments(a, S, wsum);
+  grid.sync();
+  uint64_t wins = 0, slots = 0;
+  while (true) {
+    const uint32_t done = *(volatile uint32_t *)&S.done;
+    if (done) break;
+    const uint32_t lvl = *(volatile uint32_t *)&S.lvl, q = *(volatile uint32_t *)&S.q;
+    const uint32_t cur = *(volatile uint32_t *)&S.cur;
+    const uint32_t *pt = a.pt[cur];
+    // CountSegment + CountUpdatesInSegment + density test: a warp per window
+    {
+      const int lane = threadIdx.x & 31;
+      const uint64_t nwarps = (uint64_t)gridDim.x * (CL_T / 32);
+      const uint64_t Lc = 1ull << lvl;
+      for (uint64_t w = (blockIdx.x * (uint64_t)CL_T + threadIdx.x) / 32; w < q; w += nwarps) {
+        const uint64_t leaf0 = ((uint64_t)(pt[a.wfirst[w]] >> lvl)) << lvl;
+        uint64_t n = 0;
+        for (uint64_t l = lane; l < Lc; l += 32) n += a.cnt[leaf0 + l];
+        for (int o = 16; o; o >>= 1) n += __shfl_xor_sync(0xffffffffu, n, o);
+        if (lane == 0) {
+          const uint64_t u = a.wfirst[w + 1] - a.wfirst[w];
+          const bool ok = a.op == GPMA_INSERT ? n + u <= a.tmax[lvl] : (n >= u && n - u >= a.tmin[lvl]);
+          a.acc[w] = ok ? 1u : 0u;
+          a.nw[w] = ok ? (a.op == GPMA_INSERT ? n + u : n - u) : 0;
+        }
+      }
+    }
+    grid.sync();
+    // Merge + re-dispatch evenly: a CTA per accepted window
+    for (uint32_t w = blockIdx.x; w < q; w += gridDim.x) {
+      if (!a.acc[w]) continue;
+      cl_merge_window(a, S, w, mk, mv, lpre);
+      ++wins;
+      slots += (uint64_t)a.L << lvl;
+    }
+    grid.sync();
+    if (blockIdx.x == 0) {
+      cl_promote(a, S, wsum);
+      if (!S.done) cl_segments(a, S, wsum);
+    }
+    grid.sync();
+  }
+  if (threadIdx.x == 0 && wins) {
+    atomicAdd((unsigned long long *)&S.windows, (unsigned long long)wins);
+    atomicAdd((unsigned long long *)&S.slots, (unsigned long long)slots);
+  }
+}
+
 // Whole-array even layout of a dense sorted list (create, resize; R7 over all leaves).
 __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *__restrict__ wv,
                               uint64_t N, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
@@ -2356,6 +2659,87 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   return recompute_heads(g, s);
 }
 
+// ---- the device-resident level loop from the host
+__global__ void k_coop_init(CoopState *st, uint64_t p, uint32_t cur, uint32_t lvl, Ctrl *c, uint64_t ndirty) {
+  st->p = p;
+  st->cur = cur;
+  st->lvl = lvl;
+  st->done = 0;
+  st->q = 0;
+  st->windows = 0;
+  st->slots = 0;
+  st->top = lvl;
+  c->ndirty = ndirty;
+}
+
+// GPMA_LVL_COOP=0 disables the device-resident level loop (read per call)
+static bool coop_eligible(gpma *g, uint64_t p, uint32_t lvl) {
+  const char *e = getenv("GPMA_LVL_COOP");
+  if (e && atoi(e) == 0) return false;
+  return p <= CL_MAXP && ((uint64_t)g->L << lvl) <= CL_MAXS && g->h < 48;
+}
+
+static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, uint64_t *dirty_base, int op,
+                               cudaStream_t s) {
+  const size_t smem = (size_t)CL_MAXS * 12 + 260 * 4;
+  static int blocks_per_sm = [] {
+    cudaFuncSetAttribute(k_levels_coop, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)((size_t)CL_MAXS * 12 + 260 * 4));
+    int b = 0;
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_levels_coop, CL_T, (size_t)CL_MAXS * 12 + 260 * 4);
+    return b > 0 ? b : 1;
+  }();
+  GP_CHECK(g, ensure(g, g->b_misc2, sizeof(CoopState) + 64, s));
+  CoopArgs a{};
+  for (int i = 0; i < 2; ++i) {
+    a.pk[i] = (uint64_t *)g->b_pk[i].p;
+    a.pv[i] = (uint32_t *)g->b_pv[i].p;
+    a.pt[i] = (uint32_t *)g->b_pt[i].p;
+  }
+  a.hf = (uint32_t *)g->b_hf.p;
+  a.widx = (uint32_t *)g->b_widx.p;
+  a.wfirst = (uint32_t *)g->b_wfirst.p;
+  a.acc = (uint32_t *)g->b_acc.p;
+  a.keep = (uint32_t *)g->b_keep2.p;
+  a.kpos = (uint32_t *)g->b_kpos.p;
+  a.nw = (uint64_t *)g->b_nw.p;
+  a.key = g->key;
+  a.val = g->val;
+  a.cnt = g->cnt;
+  a.tmask = tmask_of(g);
+  a.row_offset = g->row_offset;
+  a.dirty = (uint2 *)g->b_dirty.p;
+  a.nleaves = g->cap / g->L;
+  a.L = g->L;
+  a.h = g->h;
+  a.rb = g->rb;
+  a.op = op;
+  for (uint32_t i = 0; i <= g->h; ++i) {
+    a.tmin[i] = g->tmin[i];
+    a.tmax[i] = g->tmax[i];
+  }
+  a.st = (CoopState *)g->b_misc2.p;
+  a.c = g->ctrl_d;
+  GP_LAUNCH(g, k_coop_init, 1, 1, 0, s, a.st, p, (uint32_t)cur, lvl, g->ctrl_d, *dirty_base);
+  const int grid = std::max(1, std::min(blocks_per_sm * num_sms(), 4 * num_sms()));
+  void *args[] = {&a};
+  g->launches++;
+  GP_CHECK(g, cudaLaunchCooperativeKernel((void *)k_levels_coop, grid, CL_T, args, smem, s));
+  static_assert(sizeof(CoopState) <= 192, "pinned scratch");
+  GP_CHECK(g, readback(g, g->pin, a.st, sizeof(CoopState), s));
+  GP_CHECK(g, readback(g, &g->ctrl_h->ndirty, &g->ctrl_d->ndirty, 8, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  CoopState S;
+  memcpy(&S, g->pin, sizeof S);
+  g->last.last_slots_rewritten += S.slots;
+  g->last.last_windows_rewritten += S.windows;
+  if (S.top > g->last.last_top_level) g->last.last_top_level = S.top;
+  *dirty_base = g->ctrl_h->ndirty;
+  cur = (int)S.cur;
+  p = S.p;
+  lvl = S.lvl;
+  return GPMA_OK;
+}
+
 // ---- GPMA lock-based insertion (Alg. 1) -----------------------------------------------
 __global__ void k_count_leaf_live(const uint32_t *__restrict__ cnt, uint64_t nl, uint64_t *__restrict__ out) {
   for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nl;
@@ -2941,6 +3325,9 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
     }
     p = p_new;
     lvl = 1;
+  }
+  if (p > 0 && lvl >= 1 && lvl <= g->h && !g->trace_on && coop_eligible(g, p, lvl)) {
+    if ((st = coop_levels(g, cur, p, lvl, &dirty_base, op, s))) return st;
   }
   for (; lvl <= g->h && p > 0; ++lvl) {
     Lvl a = make_lvl(g, cur, p, lvl, op);

@@ -144,7 +144,8 @@ def test_config0_sliding_window_graph_replay(seed):
 
 
 @pytest.mark.parametrize("knob", ["GPMA_DEL_SORT=1", "GPMA_INS_FUSED=0", "GPMA_INS_LEAFSORT=0",
-                                  "GPMA_INS_LEAFSORT=0,GPMA_INS_THREAD=0"])
+                                  "GPMA_INS_LEAFSORT=0,GPMA_INS_THREAD=0", "GPMA_LVL_COOP=0", "GPMA_ILP=1",
+                                  "GPMA_ILP=4"])
 @pytest.mark.parametrize("seed", range(3))
 def test_config0_alternative_paths(seed, knob, monkeypatch):
     """The strategy switches (sorted lazy delete; separate pre-pass + k_level0; key-sorted fused
@@ -291,19 +292,30 @@ def test_medium_rmat_multi_tile(mode):
     assert_pr_close(x32, xo, fp64=False, what="rmat-s16 fp32")
 
 
-def test_sorted_stream_hot_window():
-    """Ascending-key batches concentrated in one region (NEXT-4 pattern): deep climbs."""
+@pytest.mark.parametrize("coop", ["1", "0"])
+@pytest.mark.parametrize("mode", [0, 1])
+def test_sorted_stream_hot_window(coop, mode, monkeypatch):
+    """Ascending-key batches concentrated in one region (NEXT-4 pattern): deep climbs through the
+    device-resident level loop (coop=1: levels with windows <= 4096 slots in one cooperative
+    kernel) or the host-driven one, then strict / lazy deletes of the hot keys."""
+    monkeypatch.setenv("GPMA_LVL_COOP", coop)
     V = 4096
     rng = np.random.default_rng(11)
     k0 = _keys(rng.integers(0, V, 20000), rng.integers(0, V, 20000))
     v0 = [1] * len(k0)
-    g = Gpma.gpma_create(V, keys_t(k0), vals_t(v0))
-    o = O.Oracle(V, k0, v0)
+    g = Gpma.gpma_create(V, keys_t(k0), vals_t(v0), delete_mode=mode)
+    o = O.Oracle(V, k0, v0, delete_mode=mode)
     for b in range(6):
         ks = _keys(np.full(3000, 7 + b), np.arange(3000))
         g.insert(keys_t(ks), vals_t([b] * 3000))
         o.insert(ks, [b] * 3000)
         assert_same_layout(g, o, what=f"hot batch {b}")
+    for b in range(6):
+        ks = _keys(np.full(2500, 7 + b), np.arange(500, 3000))
+        g.delete(keys_t(ks))
+        o.delete(ks)
+        assert_same_layout(g, o, what=f"hot delete {b}")
+    assert g.gpma_stats()["resizes"] == o.stats()["resizes"]
 
 
 def test_gpma_lock_example2_on_gpu(golden):
