@@ -1433,6 +1433,115 @@ __global__ void k_lvl_gather(Lvl a, const uint64_t *__restrict__ key, const uint
   }
 }
 
+// The same gather for windows of >= GB_CHUNK slots (high levels, the root of a resize): a CTA
+// takes one 4096-slot chunk of a window, finds the key range its occupied slots span, and stages
+// the window's pending keys of that range (a contiguous run of the sorted list, found by two
+// binary searches) in shared memory, so each live slot's rank among the pending keys is a search
+// of a few shared-memory entries instead of ~log2(pending) dependent global probes (merge-path
+// split of the window merge, Alg. 4 l.26).
+constexpr int GB_T = 256, GB_I = 16, GB_CHUNK = GB_T * GB_I, GB_SP = 4096;
+__global__ void __launch_bounds__(GB_T) k_lvl_gather_big(Lvl a, const uint64_t *__restrict__ key,
+                                                          const uint32_t *__restrict__ val, uint64_t nchunks) {
+  __shared__ uint64_t sp[GB_SP];
+  __shared__ uint64_t red_min[GB_T / 32], red_max[GB_T / 32];
+  __shared__ uint64_t s_pa, s_pb;
+  const uint32_t nacc = a.aidx[a.p];
+  const uint32_t lgw = (uint32_t)(__ffs(a.L) - 1) + a.lvl;       // window slots = 2^lgw
+  const uint64_t cpw = (1ull << lgw) / GB_CHUNK;                  // chunks per window
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint32_t leafmask = (a.L == 32 ? 0xffffffffu : ((1u << a.L) - 1u) << (lane & ~(a.L - 1)));
+  for (uint64_t ch = blockIdx.x; ch < nchunks; ch += gridDim.x) {   // block-uniform
+    const uint64_t ai = ch / cpw;
+    if (ai >= nacc) break;
+    const uint32_t w = a.alist[ai];
+    const uint64_t seg = a.pt[a.wfirst[w]] >> a.lvl;
+    const uint64_t off0 = (ch % cpw) * GB_CHUNK;                  // chunk offset in the window
+    const uint64_t s0 = seg * (1ull << lgw) + off0;
+    uint64_t k[GB_I];
+    uint32_t v[GB_I];
+    uint64_t kmin = KEY_NONE, kmax = 0;
+    bool anyocc = false;
+#pragma unroll
+    for (int i = 0; i < GB_I; ++i) {
+      const uint64_t s = s0 + (uint64_t)i * GB_T + threadIdx.x;
+      k[i] = key[s];
+      v[i] = val[s];
+      if (k[i] != KEY_NONE) {
+        kmin = min(kmin, k[i]);
+        kmax = max(kmax, k[i]);
+        anyocc = true;
+      }
+    }
+    for (int o = 16; o; o >>= 1) {
+      kmin = min(kmin, __shfl_xor_sync(0xffffffffu, kmin, o));
+      kmax = max(kmax, __shfl_xor_sync(0xffffffffu, kmax, o));
+    }
+    anyocc = __any_sync(0xffffffffu, anyocc);
+    if (lane == 0) {
+      red_min[warp] = kmin;
+      red_max[warp] = anyocc ? kmax : 0;
+    }
+    __syncthreads();
+    const uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
+    if (threadIdx.x == 0) {
+      uint64_t mn = KEY_NONE, mx = 0;
+      for (int q = 0; q < GB_T / 32; ++q) {
+        mn = min(mn, red_min[q]);
+        mx = max(mx, red_max[q]);
+      }
+      uint64_t pa = ub, pb = ub;
+      if (mn != KEY_NONE) {
+        pa = lower_bound_u64(a.pk, ub, ue, mn);
+        pb = lower_bound_u64(a.pk, pa, ue, mx == KEY_NONE ? mx : mx + 1);
+      }
+      s_pa = pa;
+      s_pb = pb;
+    }
+    __syncthreads();
+    const uint64_t pa = s_pa, pb = s_pb;
+    const bool staged = pb - pa <= (uint64_t)GB_SP;
+    if (staged)
+      for (uint64_t j = pa + threadIdx.x; j < pb; j += GB_T) sp[j - pa] = a.pk[j];
+    __syncthreads();
+#pragma unroll
+    for (int i = 0; i < GB_I; ++i) {
+      const uint64_t off = off0 + (uint64_t)i * GB_T + threadIdx.x;     // slot offset in the window
+      const bool live = k[i] != KEY_NONE && v[i] != VAL_TOMB;
+      const uint32_t bal = __ballot_sync(0xffffffffu, live);
+      if (!live) continue;
+      const uint64_t lidx = leaf_div(off, a.L);
+      const uint64_t rl = __popc(bal & leafmask & lt) + (a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl]);
+      uint64_t c;                                        // pending keys < k[i] in the window
+      if (staged) {
+        uint64_t lo = 0, hi = pb - pa;
+        while (lo < hi) {
+          const uint64_t mid = (lo + hi) >> 1;
+          if (sp[mid] < k[i]) lo = mid + 1;
+          else hi = mid;
+        }
+        c = pa - ub + lo;
+      } else {
+        c = lower_bound_u64(a.pk, pa, pb, k[i]) - ub;
+      }
+      uint64_t r;
+      bool drop = false;
+      if (a.op == GPMA_INSERT) {
+        r = rl + c;
+      } else {
+        drop = (ub + c < ue) && a.pk[ub + c] == k[i];
+        r = rl - c;
+      }
+      if (!drop) {
+        const uint64_t d = a.woff[w] + r;
+        a.wk[d] = k[i];
+        a.wv[d] = v[i];
+      }
+    }
+    __syncthreads();                                     // sp / red reused by the next chunk
+  }
+}
+
 // Place the pending insertions of accepted windows at their merged rank.
 __global__ void k_lvl_place(Lvl a, const uint64_t *__restrict__ key, const uint32_t *__restrict__ val) {
   for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < a.p;
@@ -1915,7 +2024,7 @@ __device__ void cl_merge_window(const CoopArgs &a, const CoopState &S, uint32_t 
   const int lane = threadIdx.x & 31;
   const uint32_t lt = (1u << lane) - 1u;
   const uint32_t leafmask = (L == 32 ? 0xffffffffu : ((1u << L) - 1u) << (lane & ~(L - 1)));
-  // live entries before each leaf of the window (Lc <= 256)
+  // live entries before each leaf of the window (Lc <= CL_MAXS / 4)
   if (threadIdx.x < 32) {
     uint32_t carry = 0;
     for (uint32_t l0 = 0; l0 < Lc; l0 += 32) {
@@ -2010,7 +2119,7 @@ __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
   extern __shared__ __align__(16) unsigned char cl_smem[];
   uint64_t *mk = reinterpret_cast<uint64_t *>(cl_smem);
   uint32_t *mv = reinterpret_cast<uint32_t *>(mk + CL_MAXS);
-  uint32_t *lpre = mv + CL_MAXS;                         // [257]
+  uint32_t *lpre = mv + CL_MAXS;                         // [CL_MAXS / 4 + 1] (L >= 4)
   __shared__ uint64_t wsum[CL_T / 32];
   cooperative_groups::grid_group grid = cooperative_groups::this_grid();
   CoopState &S = *a.st;
@@ -2062,28 +2171,36 @@ __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
   }
 }
 
-// Whole-array even layout of a dense sorted list (create, resize; R7 over all leaves).
+// Whole-array even layout of a dense sorted list (create, resize; R7 over all leaves): a thread
+// writes 4 consecutive slots of one leaf with 16-B stores (two key pairs, one value quad).
 __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *__restrict__ wv,
                               uint64_t N, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
                               uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset,
                               uint32_t L, uint64_t nleaves, uint32_t rb) {
   uint32_t *tmask = cnt + nleaves;
   const uint64_t cap = nleaves * L;
-  for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < cap;
-       s += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t l = leaf_div(s, L), p = leaf_mod(s, L);
-    uint64_t lo = l * N / nleaves, hi = (l + 1) * N / nleaves;
-    if (p < hi - lo) {
-      uint64_t k = wk[lo + p];
-      key[s] = k;
-      val[s] = wv[lo + p];
-      if (is_guard_key(k)) row_offset[(k >> 32) - rb + 1] = s;
-    } else {
-      key[s] = KEY_NONE;
-      val[s] = 0;
+  for (uint64_t s = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) * 4; s < cap;
+       s += (uint64_t)gridDim.x * blockDim.x * 4) {
+    const uint64_t l = leaf_div(s, L), p = leaf_mod(s, L);
+    const uint64_t lo = l * N / nleaves, hi = (l + 1) * N / nleaves, m = hi - lo;
+    uint64_t k[4];
+    uint32_t v[4];
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      if (p + q < m) {
+        k[q] = wk[lo + p + q];
+        v[q] = wv[lo + p + q];
+        if (is_guard_key(k[q])) row_offset[(k[q] >> 32) - rb + 1] = s + q;
+      } else {
+        k[q] = KEY_NONE;
+        v[q] = 0;
+      }
     }
+    *reinterpret_cast<ulonglong2 *>(key + s) = make_ulonglong2(k[0], k[1]);
+    *reinterpret_cast<ulonglong2 *>(key + s + 2) = make_ulonglong2(k[2], k[3]);
+    *reinterpret_cast<uint4 *>(val + s) = make_uint4(v[0], v[1], v[2], v[3]);
     if (p == 0) {
-      cnt[l] = (uint32_t)(hi - lo);
+      cnt[l] = (uint32_t)m;
       tmask[l] = 0u;
       uint32_t gc = 0;
       for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(wk[e]);
@@ -2287,7 +2404,7 @@ static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v
 gpma_status build_from_sorted(gpma *g, const uint64_t *wk, const uint32_t *wv, uint64_t N,
                               cudaStream_t s) {
   uint64_t nl = g->cap / g->L;
-  GP_LAUNCH(g, k_layout_even, grid_for(g->cap), TB, 0, s, wk, wv, N, g->key, g->val, g->cnt,
+  GP_LAUNCH(g, k_layout_even, grid_for(g->cap / 4), TB, 0, s, wk, wv, N, g->key, g->val, g->cnt,
             g->row_offset, g->L, nl, g->rb);
   GP_CHECK(g, cudaGetLastError());
   gpma_status st = recompute_heads(g, s);
@@ -2446,6 +2563,12 @@ static int lvl_small_on() {      // 0 off, 1 front/back only, 2 (default) + fuse
   return e ? atoi(e) : 2;
 }
 
+// GPMA_GATHER_BIG=0: windows of >= 4096 slots gathered by the per-slot global search instead
+static bool gather_big_on() {
+  const char *e = getenv("GPMA_GATHER_BIG");
+  return !e || atoi(e) != 0;
+}
+
 static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t *dirty_base,
                               cudaStream_t s, bool resize_target, uint64_t new_cap, uint64_t *nk,
                               uint32_t *nv, uint32_t *ncnt) {
@@ -2498,7 +2621,13 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     }
     uint64_t bslots = wins_bound * wslots;
     uint64_t bslots_r = (bslots + 31) & ~31ull;
-    GP_LAUNCH(g, k_lvl_gather, grid_for(bslots_r), TB, 0, s, a, g->key, g->val, bslots_r);
+    if (a.lvl && wslots >= (uint64_t)GB_CHUNK && gather_big_on()) {
+      const uint64_t nch = bslots / GB_CHUNK;
+      GP_LAUNCH(g, k_lvl_gather_big, (unsigned)std::min<uint64_t>(nch, (uint64_t)num_sms() * 8), GB_T, 0, s, a, g->key,
+                g->val, nch);
+    } else {
+      GP_LAUNCH(g, k_lvl_gather, grid_for(bslots_r), TB, 0, s, a, g->key, g->val, bslots_r);
+    }
     if (a.op == GPMA_INSERT) GP_LAUNCH(g, k_lvl_place, gp, TB, 0, s, a, g->key, g->val);
     if (!resize_target) {
       GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots), TB, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
@@ -2510,7 +2639,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
       GP_CHECK(g, cudaStreamSynchronize(s));
       N = g->ctrl_h->sum;
       uint64_t nl_new = new_cap / g->L;
-      GP_LAUNCH(g, k_layout_even, grid_for(new_cap), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
+      GP_LAUNCH(g, k_layout_even, grid_for(new_cap / 4), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
                 g->row_offset, g->L, nl_new, g->rb);
     }
   }
@@ -2681,11 +2810,11 @@ static bool coop_eligible(gpma *g, uint64_t p, uint32_t lvl) {
 
 static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, uint64_t *dirty_base, int op,
                                cudaStream_t s) {
-  const size_t smem = (size_t)CL_MAXS * 12 + 260 * 4;
+  constexpr size_t smem = (size_t)CL_MAXS * 12 + (CL_MAXS / 4 + 4) * 4;
   static int blocks_per_sm = [] {
-    cudaFuncSetAttribute(k_levels_coop, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)((size_t)CL_MAXS * 12 + 260 * 4));
+    cudaFuncSetAttribute(k_levels_coop, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     int b = 0;
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_levels_coop, CL_T, (size_t)CL_MAXS * 12 + 260 * 4);
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_levels_coop, CL_T, smem);
     return b > 0 ? b : 1;
   }();
   GP_CHECK(g, ensure(g, g->b_misc2, sizeof(CoopState) + 64, s));
@@ -2861,7 +2990,7 @@ static gpma_status double_root(gpma *g, cudaStream_t s) {
   uint32_t *nv, *ncnt;
   uint64_t *nhead;
   if ((st = alloc_store(g, cap2, &nk, &nv, &ncnt, &nhead, s))) return st;
-  GP_LAUNCH(g, k_layout_even, grid_for(cap2), TB, 0, s, (const uint64_t *)g->b_wk.p, (const uint32_t *)g->b_wv.p,
+  GP_LAUNCH(g, k_layout_even, grid_for(cap2 / 4), TB, 0, s, (const uint64_t *)g->b_wk.p, (const uint32_t *)g->b_wv.p,
             N, nk, nv, ncnt, g->row_offset, g->L, cap2 / g->L, g->rb);
   dev_free(g, g->key, s);
   dev_free(g, g->val, s);
