@@ -690,6 +690,120 @@ __global__ void k_gflags(const uint64_t *__restrict__ tk, uint64_t n, uint32_t *
 // (R11, R12); the rest are new -- and writes keep[j] = 1 for the new ones.  Accepted (density
 // n_live + u_new <= max_0): tombstones dropped, the new keys inserted at their key rank (one
 // static shift each, any order), the leaf written back; rejected: hits in place, keep stays 1.
+// ---- one leaf group, the leaf in a row of shared memory (rk, rv): Alg. 4 l.3-15 at the leaves
+// for the updates j0..j1 of the group (any order; U.key(j) / U.val(j)).  The last copy of a key
+// in the group acts (R10); a key equal to an occupied slot overwrites (R11) / revives (R12) it;
+// the rest are new.  Density n_live + u_new <= max_0 (l.25, R5): the tombstones are dropped,
+// the new keys inserted at their key rank, the row left-packed (R7 for one leaf) and the leaf's
+// count / tombstone mask / head / guard row offsets maintained; otherwise the hits stay in
+// place and keep[j] = 1 flags the new keys pending for level 1.  Out-degrees: +1 per new key
+// or revive.  The caller writes the row back (keys when ok, values when ok or hitm).
+struct LeafOut {
+  bool ok = false;
+  uint32_t hitm = 0, nnew = 0, effs = 0;
+};
+
+struct UpdIdx {                 // the leaf-sorted batch: arrival indices into the staged batch
+  const uint64_t *ik;
+  const uint32_t *iv;
+  const uint32_t *tix;
+  __device__ uint64_t key(uint32_t j) const { return ik[tix[j]]; }
+  __device__ uint32_t val(uint32_t j) const { return iv[tix[j]]; }
+};
+
+struct UpdDirect {              // a key-sorted batch (shared or global memory)
+  const uint64_t *k;
+  const uint32_t *v;
+  __device__ uint64_t key(uint32_t j) const { return k[j]; }
+  __device__ uint32_t val(uint32_t j) const { return v[j]; }
+};
+
+template <class Upd>
+__device__ __forceinline__ LeafOut leaf_group_merge(uint64_t *rk, uint32_t *rv, uint32_t L, uint32_t t, uint32_t j0,
+                                                    uint32_t j1, const Upd &U, uint32_t bound, uint32_t *keep,
+                                                    const uint64_t *key, uint32_t *cnt, uint32_t *tmask,
+                                                    uint64_t *head, uint64_t *row_offset, uint32_t *deg, uint32_t rb,
+                                                    uint2 *dirty, Ctrl *c) {
+  LeafOut o;
+  const uint64_t lb = (uint64_t)t * L;
+  uint32_t nocc = 0, tomb = 0;
+  for (; nocc < L && rk[nocc] != KEY_NONE; ++nocc) tomb |= (rv[nocc] == VAL_TOMB ? 1u : 0u) << nocc;
+  const uint64_t h_old = rk[0];
+  uint32_t revm = 0;
+  for (uint32_t j = j0; j < j1; ++j) {
+    const uint64_t uk = U.key(j);
+    bool last = true;                                    // R10: a later copy in the group wins
+    for (uint32_t j2 = j + 1; j2 < j1 && last; ++j2) last = U.key(j2) != uk;
+    uint32_t h = 0;
+    if (last) {
+      ++o.effs;
+      uint32_t lo = 0, hi = nocc;                        // the occupied prefix is sorted
+      while (lo < hi) {
+        const uint32_t mid = (lo + hi) >> 1;
+        if (rk[mid] < uk) lo = mid + 1;
+        else hi = mid;
+      }
+      if (lo < nocc && rk[lo] == uk) {                   // overwrite (R11) / revive (R12)
+        h = 1u << lo;
+        rv[lo] = U.val(j);
+      }
+      o.hitm |= h;
+      revm |= h & tomb;
+      o.nnew += h ? 0u : 1u;
+      if (!h || (h & tomb)) atomicAdd(&deg[(uint32_t)(uk >> 32) - rb], 1u);   // new key or revive
+    }
+    keep[j] = (last && !h) ? 1u : 0u;
+  }
+  const uint32_t dead = tomb & ~revm;
+  const uint32_t n = nocc - __popc(dead);
+  o.ok = o.nnew > 0 && o.nnew <= bound && n + o.nnew <= bound;
+  if (o.ok) {
+    uint32_t N = n;
+    if (dead) {                                          // drop the tombstones: left-pack the live
+      uint32_t w2 = 0;
+      for (uint32_t p = 0; p < nocc; ++p)
+        if (!((dead >> p) & 1u)) {
+          rk[w2] = rk[p];
+          rv[w2] = rv[p];
+          ++w2;
+        }
+    }
+    for (uint32_t j = j0; j < j1; ++j) {                 // the new keys at their key rank
+      if (!keep[j]) continue;
+      keep[j] = 0u;
+      const uint64_t uk = U.key(j);
+      uint32_t pos = N;
+      while (pos > 0 && rk[pos - 1] > uk) {
+        rk[pos] = rk[pos - 1];
+        rv[pos] = rv[pos - 1];
+        --pos;
+      }
+      rk[pos] = uk;
+      rv[pos] = U.val(j);
+      ++N;
+    }
+    for (uint32_t p = N; p < nocc; ++p) {
+      rk[p] = KEY_NONE;
+      rv[p] = 0;
+    }
+    for (uint32_t p = 0; p < N; ++p)
+      if (is_guard_key(rk[p])) row_offset[(rk[p] >> 32) - rb + 1] = lb + p;   // R8: guards that moved
+    cnt[t] = N;
+    if (tomb) tmask[t] = 0u;                             // (no tombstone in the leaf: already 0)
+    if (rk[0] != h_old) {
+      head[t] = rk[0];
+      if (t > 0 && key[lb - L] == KEY_NONE) {            // empty leaves to the left carry this head
+        const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
+        dirty[d] = make_uint2(t, 1u);
+      }
+    }
+  } else if (revm) {
+    cnt[t] += __popc(revm);
+    tmask[t] &= ~revm;
+  }
+  return o;
+}
+
 constexpr int ILU_T = 128;      // 4 warps: 4 x 32 leaves staged in shared memory
 template <int L>
 __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
@@ -755,89 +869,15 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
     __syncwarp();
     // the thread's leaf is its row of shared memory: dynamic indexing is free there, so the
     // merge is a few moves per update instead of static select networks over registers
-    uint64_t *const rk = mk + lane * KS;
-    uint32_t *const rv = mv + lane * KS;
-    uint32_t nocc = 0, tomb = 0;
-    if (have) {
-      for (; nocc < (uint32_t)L && rk[nocc] != KEY_NONE; ++nocc) tomb |= (rv[nocc] == VAL_TOMB ? 1u : 0u) << nocc;
-    }
-    const uint64_t h_old = have ? rk[0] : KEY_NONE;
-    uint32_t hitm = 0, revm = 0, nnew = 0;
-    for (uint32_t j = j0; j < j1; ++j) {
-      const uint32_t i = tix[j];
-      const uint64_t uk = ik[i];
-      bool last = true;                                  // R10: a later copy in the group wins
-      for (uint32_t j2 = j + 1; j2 < j1 && last; ++j2) last = ik[tix[j2]] != uk;
-      uint32_t h = 0;
-      if (last) {
-        ++effs;
-        uint32_t lo = 0, hi = nocc;                      // the occupied prefix is sorted
-        while (lo < hi) {
-          const uint32_t mid = (lo + hi) >> 1;
-          if (rk[mid] < uk) lo = mid + 1;
-          else hi = mid;
-        }
-        if (lo < nocc && rk[lo] == uk) {                 // overwrite (R11) / revive (R12)
-          h = 1u << lo;
-          rv[lo] = iv[i];
-        }
-        hitm |= h;
-        revm |= h & tomb;
-        nnew += h ? 0u : 1u;
-        if (!h || (h & tomb)) atomicAdd(&deg[(uint32_t)(uk >> 32) - rb], 1u);   // new key or revive
-      }
-      keep[j] = (last && !h) ? 1u : 0u;
-    }
-    const uint32_t dead = tomb & ~revm;
-    const uint32_t n = nocc - __popc(dead);
-    const bool ok = have && nnew > 0 && nnew <= bound && n + nnew <= bound;
-    news += nnew;
-    if (ok) {
-      uint32_t N = n;
-      if (dead) {                                        // drop the tombstones: left-pack the live
-        uint32_t w2 = 0;
-        for (uint32_t p = 0; p < nocc; ++p)
-          if (!((dead >> p) & 1u)) {
-            rk[w2] = rk[p];
-            rv[w2] = rv[p];
-            ++w2;
-          }
-      }
-      for (uint32_t j = j0; j < j1; ++j) {               // the new keys at their key rank
-        if (!keep[j]) continue;
-        keep[j] = 0u;
-        const uint32_t i = tix[j];
-        const uint64_t uk = ik[i];
-        uint32_t pos = N;
-        while (pos > 0 && rk[pos - 1] > uk) {
-          rk[pos] = rk[pos - 1];
-          rv[pos] = rv[pos - 1];
-          --pos;
-        }
-        rk[pos] = uk;
-        rv[pos] = iv[i];
-        ++N;
-      }
-      for (uint32_t p = N; p < nocc; ++p) {
-        rk[p] = KEY_NONE;
-        rv[p] = 0;
-      }
-      for (uint32_t p = 0; p < N; ++p)
-        if (is_guard_key(rk[p])) row_offset[(rk[p] >> 32) - rb + 1] = lb + p;   // R8: guards that moved
-      cnt[t] = N;
-      if (tomb) tmask[t] = 0u;                          // (no tombstone in the leaf: already 0)
-      if (rk[0] != h_old) {
-        head[t] = rk[0];
-        if (t > 0 && key[lb - L] == KEY_NONE) {          // empty leaves to the left carry this head
-          const uint64_t d = atomicAdd((unsigned long long *)&c->ndirty, 1ull);
-          dirty[d] = make_uint2(t, 1u);
-        }
-      }
-      ++accepted;
-    } else if (have && revm) {
-      cnt[t] += __popc(revm);
-      tmask[t] &= ~revm;
-    }
+    const UpdIdx U{ik, iv, tix};
+    const LeafOut lo_ = have ? leaf_group_merge(mk + lane * KS, mv + lane * KS, (uint32_t)L, t, j0, j1, U, bound, keep,
+                                                key, cnt, tmask, head, row_offset, deg, rb, dirty, c)
+                             : LeafOut{};
+    const bool ok = lo_.ok;
+    const uint32_t hitm = lo_.hitm;
+    news += lo_.nnew;
+    effs += lo_.effs;
+    accepted += ok ? 1u : 0u;
     const bool vdirty = ok || hitm;                      // the values go back for hits too
     __syncwarp();
     // cooperative store of the accepted (rewritten) leaves
@@ -867,6 +907,239 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
     if (accepted) atomicAdd((unsigned long long *)&c->windows_rewritten, (unsigned long long)accepted);
     if (news) atomicAdd((unsigned long long *)&c->sum, (unsigned long long)news);
     if (effs) atomicAdd((unsigned long long *)&c->nunique, (unsigned long long)effs);
+  }
+}
+
+// ---- small batches in ONE kernel (n <= SB_MAX): the paper names kernel-call overheads as what
+// dominates small batches.  A single CTA validates the batch (nothing changes on
+// an error), sorts it by key in shared memory (bitonic, arrival index breaks ties: stable, R10),
+// locates every key (R9), forms the leaf groups, merges them (leaf_group_merge, leaves staged
+// in shared-memory rows), compacts the rejected keys -- already key-sorted -- into the pending
+// list for level 1 and mirrors its control block to pinned host memory: one launch and one
+// host synchronisation per call instead of a dozen launches.  Lazy deletes likewise.
+constexpr int SB_T = 1024, SB_MAX = 2048, SB_ROWS = 256, SB_DEL_MAX = 4096;
+constexpr size_t SB_ROWK_OFF = ((size_t)SB_MAX * 8 + (size_t)SB_MAX * 4 * 2 + (size_t)(SB_MAX + 1) * 4 * 2 + 15) & ~(size_t)15;
+__host__ __device__ constexpr size_t sb_smem_bytes(int L) { return SB_ROWK_OFF + (size_t)SB_ROWS * (L + 1) * 12; }
+
+__device__ __forceinline__ void sb_block_scan2(uint32_t (&v)[2], uint32_t *wsum, uint32_t *total) {
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint32_t t = v[0] + v[1];
+  uint32_t x = t;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if (lane >= o) x += y;
+  }
+  if (lane == 31) wsum[warp] = x;
+  __syncthreads();
+  if (warp == 0) {
+    uint32_t w = wsum[lane];
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, w, o);
+      if (lane >= o) w += y;
+    }
+    wsum[lane] = w;
+  }
+  __syncthreads();
+  const uint32_t base = (warp ? wsum[warp - 1] : 0) + x - t;
+  *total = wsum[31];
+  __syncthreads();
+  v[1] = base + v[0];
+  v[0] = base;
+}
+
+template <int L>
+__global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
+                                                       uint32_t n, uint64_t *key, uint32_t *val, uint32_t *cnt,
+                                                       uint32_t *tmask, uint64_t *head, uint64_t *row_offset,
+                                                       uint32_t *deg, uint32_t nleaves, uint32_t rb, uint32_t nr,
+                                                       uint32_t V, uint32_t bound, const uint64_t *__restrict__ ro,
+                                                       uint64_t *pk, uint32_t *pv, uint32_t *pt, uint2 *dirty, Ctrl *c,
+                                                       Ctrl *c_host) {
+  extern __shared__ __align__(16) unsigned char sb_smem[];
+  uint64_t *sk = reinterpret_cast<uint64_t *>(sb_smem);           // [SB_MAX] keys (sorted)
+  uint32_t *si = reinterpret_cast<uint32_t *>(sk + SB_MAX);       // [SB_MAX] arrival index -> sorted values
+  uint32_t *st = si + SB_MAX;                                     // [SB_MAX] target leaves
+  uint32_t *kp = st + SB_MAX;                                     // [SB_MAX + 1] keep flags / group starts
+  uint32_t *gs = kp + SB_MAX + 1;                                 // [SB_MAX + 1] group starts
+  uint64_t *rowk = reinterpret_cast<uint64_t *>(sb_smem + SB_ROWK_OFF);   // [SB_ROWS][L + 1]
+  uint32_t *rowv = reinterpret_cast<uint32_t *>(rowk + SB_ROWS * (L + 1));
+  __shared__ uint32_t wsum[32];
+  __shared__ uint32_t s_stats[3];
+  const int tid = threadIdx.x;
+  if (tid == 0) {
+    c->err = 0;
+    c->nunique = 0;
+    c->windows_rewritten = 0;
+    c->ndirty = 0;
+    c->sum = 0;
+    c->sum2 = 0;
+    s_stats[0] = s_stats[1] = s_stats[2] = 0;
+  }
+  // validate (RESERVED beats RANGE; nothing is mutated on either)
+  uint32_t e = 0;
+  for (uint32_t i = tid; i < n; i += SB_T) {
+    const uint64_t k = ik[i];
+    const uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
+    if (dst == COL_GUARD || iv[i] == VAL_TOMB) e |= 2u;
+    if (src - rb >= nr || dst >= V) e |= 1u;
+  }
+  e = __syncthreads_or(e) ? (__reduce_or_sync(0xffffffffu, e)) : 0u;
+  if (e) atomicOr(&c->err, e);
+  __syncthreads();
+  if (c->err) {
+    if (tid == 0) *c_host = *c;
+    return;
+  }
+  // stable sort by key (bitonic over the next power of two; the arrival index breaks ties)
+  uint32_t np2 = 1;
+  while (np2 < n) np2 <<= 1;
+  for (uint32_t i = tid; i < np2; i += SB_T) {
+    sk[i] = i < n ? ik[i] : KEY_NONE;
+    si[i] = i;
+  }
+  __syncthreads();
+  for (uint32_t size = 2; size <= np2; size <<= 1)
+    for (uint32_t stride = size >> 1; stride; stride >>= 1) {
+      for (uint32_t i = tid; i < np2; i += SB_T) {
+        const uint32_t j = i ^ stride;
+        if (j > i) {
+          const bool up = (i & size) == 0;
+          const bool gt = sk[i] > sk[j] || (sk[i] == sk[j] && si[i] > si[j]);
+          if (gt == up) {
+            const uint64_t tk = sk[i];
+            sk[i] = sk[j];
+            sk[j] = tk;
+            const uint32_t ti = si[i];
+            si[i] = si[j];
+            si[j] = ti;
+          }
+        }
+      }
+      __syncthreads();
+    }
+  // values in key order, targets (R9), group heads
+  uint32_t f[2];
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    f[q] = 0;
+    if (i < n) {
+      si[i] = iv[si[i]];
+      st[i] = locate_leaf_rows(head, nleaves, ro, rb, L, sk[i]);
+    }
+  }
+  __syncthreads();
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    f[q] = (i < n && (i == 0 || st[i] != st[i - 1])) ? 1u : 0u;
+  }
+  uint32_t fe[2] = {f[0], f[1]}, ng = 0;
+  sb_block_scan2(fe, wsum, &ng);
+  for (int q = 0; q < 2; ++q)
+    if (f[q]) gs[fe[q]] = tid * 2 + q;
+  if (tid == 0) gs[ng] = n;
+  __syncthreads();
+  // the leaf groups, SB_ROWS at a time, each leaf in a shared-memory row
+  const UpdDirect U{sk, si};
+  for (uint32_t g0 = 0; g0 < ng; g0 += SB_ROWS) {
+    const uint32_t gi = g0 + tid;
+    if (tid < SB_ROWS && gi < ng) {
+      const uint32_t j0 = gs[gi], j1 = gs[gi + 1], t = st[j0];
+      const uint64_t lb = (uint64_t)t * L;
+      uint64_t *rk = rowk + tid * (L + 1);
+      uint32_t *rv = rowv + tid * (L + 1);
+      for (int p = 0; p < L; ++p) {
+        rk[p] = key[lb + p];
+        rv[p] = val[lb + p];
+      }
+      const LeafOut o = leaf_group_merge(rk, rv, (uint32_t)L, t, j0, j1, U, bound, kp, key, cnt, tmask, head,
+                                         row_offset, deg, rb, dirty, c);
+      if (o.ok)
+        for (int p = 0; p < L; ++p) key[lb + p] = rk[p];
+      if (o.ok || o.hitm)
+        for (int p = 0; p < L; ++p) val[lb + p] = rv[p];
+      atomicAdd(&s_stats[0], o.ok ? 1u : 0u);
+      atomicAdd(&s_stats[1], o.nnew);
+      atomicAdd(&s_stats[2], o.effs);
+    }
+  }
+  __syncthreads();
+  // the rejected new keys, in key order, with their targets: the pending list of level 1
+  uint32_t kf[2];
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    kf[q] = i < n ? kp[i] : 0u;
+  }
+  uint32_t kq[2] = {kf[0], kf[1]}, npend = 0;
+  sb_block_scan2(kq, wsum, &npend);
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    if (kf[q]) {
+      pk[kq[q]] = sk[i];
+      pv[kq[q]] = si[i];
+      pt[kq[q]] = st[i];
+    }
+  }
+  __syncthreads();
+  if (tid == 0) {
+    c->windows_rewritten += s_stats[0];
+    c->sum = s_stats[1];              // new keys (pending after the pre-pass, in the old terms)
+    c->nunique = s_stats[2];
+    c->sum2 = npend;                  // pending after level 0
+    __threadfence_system();
+    *c_host = *c;                     // the control block, mirrored (zero-copy) for the host
+  }
+}
+
+// small lazy-delete batch: validate, then mark, one CTA, one launch
+__global__ void __launch_bounds__(SB_T) k_small_delete(const uint64_t *__restrict__ ik, uint32_t n,
+                                                       const uint64_t *__restrict__ key, uint32_t *val, uint32_t *cnt,
+                                                       const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
+                                                       uint32_t *tmask, uint32_t *deg, uint32_t rb, uint32_t nr,
+                                                       uint32_t V, const uint64_t *__restrict__ ro, Ctrl *c,
+                                                       Ctrl *c_host) {
+  const int tid = threadIdx.x;
+  if (tid == 0) {
+    c->err = 0;
+    c->nunique = 0;
+    c->sum = 0;
+    c->sum2 = 0;
+  }
+  uint32_t e = 0;
+  for (uint32_t i = tid; i < n; i += SB_T) {
+    const uint64_t k = ik[i];
+    const uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
+    if (dst == COL_GUARD) e |= 2u;
+    if (src - rb >= nr || dst >= V) e |= 1u;
+  }
+  e = __syncthreads_or(e) ? (__reduce_or_sync(0xffffffffu, e)) : 0u;
+  if (e) atomicOr(&c->err, e);
+  __syncthreads();
+  if (!c->err) {
+    for (uint32_t i = tid; i < n; i += SB_T) {
+      const uint64_t k = ik[i];
+      const uint32_t t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
+      const uint64_t base = (uint64_t)t * L;
+      const int p = find_in_leaf(key, base, L, k);
+      if (p < 0) continue;
+      uint32_t old = val[base + p];
+      while (old != VAL_TOMB) {                          // duplicates: one of them accounts it
+        const uint32_t seen = atomicCAS(&val[base + p], old, VAL_TOMB);
+        if (seen == old) {
+          atomicSub(&cnt[t], 1u);
+          atomicOr(&tmask[t], 1u << p);
+          atomicSub(&deg[(uint32_t)(k >> 32) - rb], 1u);
+          break;
+        }
+        old = seen;
+      }
+    }
+  }
+  __syncthreads();
+  if (tid == 0) {
+    __threadfence_system();
+    *c_host = *c;
   }
 }
 
@@ -3091,7 +3364,7 @@ static bool env_on(const char *name) {
   return !e || atoi(e) != 0;
 }
 
-enum { PATH_LAZY_UNSORTED = 0, PATH_LAZY_SORTED, PATH_INS_FUSED, PATH_INS_LEAF, PATH_GENERIC };
+enum { PATH_LAZY_UNSORTED = 0, PATH_LAZY_SORTED, PATH_INS_FUSED, PATH_INS_LEAF, PATH_GENERIC, PATH_INS_SMALL };
 
 // GPMA_INS_THREAD=0: the fused insert leaf step by L-lane sub-warps (k_ins_leaf) instead of a
 // thread per leaf group (k_ins_leaf_t, L <= 16)
@@ -3267,6 +3540,50 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
   return GPMA_OK;
 }
 
+// GPMA_SMALL=0 disables the one-kernel small-batch path (read per call)
+static bool small_batch_path(gpma *g, uint64_t n, int op, int path) {
+  const char *e = getenv("GPMA_SMALL");
+  if (e && atoi(e) == 0) return false;
+  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) return n <= (uint64_t)SB_DEL_MAX;
+  if (path == PATH_INS_LEAF || path == PATH_INS_FUSED)
+    return n <= (uint64_t)SB_MAX && (g->L == 4 || g->L == 8 || g->L == 16);
+  return false;
+}
+
+static gpma_status run_small(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, int op, cudaStream_t s) {
+  const uint64_t nl = g->cap / g->L;
+  const uint64_t *ro = g->rows_indexed ? g->row_offset : nullptr;
+  if (op == GPMA_DELETE) {
+    GP_LAUNCH(g, k_small_delete, 1, SB_T, 0, s, ik, (uint32_t)n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
+              tmask_of(g), g->deg, g->rb, g->nr, g->V, ro, g->ctrl_d, g->ctrl_h);
+    GP_CHECK(g, cudaGetLastError());
+    return GPMA_OK;
+  }
+  gpma_status st;
+  if ((st = level_buffers(g, n, s))) return st;
+  static const bool attr = [] {
+    cudaFuncSetAttribute(k_small_insert<16>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sb_smem_bytes(16));
+    cudaFuncSetAttribute(k_small_insert<8>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sb_smem_bytes(8));
+    cudaFuncSetAttribute(k_small_insert<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sb_smem_bytes(4));
+    return true;
+  }();
+  (void)attr;
+  const uint32_t bound = (uint32_t)g->tmax[0];
+  uint64_t *pk = (uint64_t *)g->b_pk[0].p;
+  uint32_t *pv = (uint32_t *)g->b_pv[0].p, *pt = (uint32_t *)g->b_pt[0].p;
+  uint2 *dirty = (uint2 *)g->b_dirty.p;
+#define GP_SMALL_INS(LL)                                                                                         \
+  GP_LAUNCH(g, k_small_insert<LL>, 1, SB_T, sb_smem_bytes(LL), s, ik, iv, (uint32_t)n, g->key, g->val, g->cnt,   \
+            tmask_of(g), g->head, g->row_offset, g->deg, (uint32_t)nl, g->rb, g->nr, g->V, bound, ro, pk, pv, pt, \
+            dirty, g->ctrl_d, g->ctrl_h)
+  if (g->L == 16) GP_SMALL_INS(16);
+  else if (g->L == 8) GP_SMALL_INS(8);
+  else GP_SMALL_INS(4);
+#undef GP_SMALL_INS
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 // everything the prefix bakes into its launches
 static std::vector<uint64_t> upd_signature(gpma *g, uint64_t n, int op) {
   std::vector<uint64_t> v = {n, (uint64_t)op, (uint64_t)prefix_path(g, op), g->mode, g->algorithm, g->V, g->rb,
@@ -3378,9 +3695,14 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));
   if (op == GPMA_INSERT) GP_CHECK(g, stage_in(g, iv, vals, n * 4, s));
   const uint64_t nl = g->cap / g->L;
-  const int path = prefix_path(g, op);
+  int path = prefix_path(g, op);
   Sorted srt;
-  if ((st = run_prefix(g, ik, iv, n, op, &srt, s))) return st;
+  if (small_batch_path(g, n, op, path)) {
+    if ((st = run_small(g, ik, iv, n, op, s))) return st;
+    path = path == PATH_INS_LEAF || path == PATH_INS_FUSED ? PATH_INS_SMALL : path;
+  } else if ((st = run_prefix(g, ik, iv, n, op, &srt, s))) {
+    return st;
+  }
   GP_CHECK(g, cudaStreamSynchronize(s));             // the one host round trip of the batch
   if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) {
     g->last.last_unique = n;   // (lazy deletes are idempotent; the sorted path marks each key once)
@@ -3398,7 +3720,17 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   int cur = 0;
   uint64_t dirty_base = 0;
   uint32_t lvl = 0;
-  if (path == PATH_INS_LEAF) {
+  if (path == PATH_INS_SMALL) {
+    // the one-kernel small batch left the rejected keys key-sorted in the level-1 buffers
+    const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
+    dirty_base = g->ctrl_h->ndirty;
+    g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;
+    g->last.last_windows_rewritten += g->ctrl_h->windows_rewritten;
+    g->last.last_level0_windows = g->ctrl_h->windows_rewritten;
+    if (p_new) g->last.last_top_level = 1;
+    p = p_new;
+    lvl = 1;
+  } else if (path == PATH_INS_LEAF) {
     // pending after level 0: the new keys the leaves rejected, gathered in leaf order, then put
     // in key order (the level loop's pending lists are key-sorted, Alg. 4 l.12-15)
     const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
