@@ -874,6 +874,107 @@ __global__ void __launch_bounds__(TA) k_pr_push_win(const uint64_t *__restrict__
   }
 }
 
+// Split push (GPMA_PR_SPLIT=1): y is just larger than L2 (8 B x 2^24 = 128 MB vs 126 MB), so
+// its REDs miss (RED-bound, not HBM-bound).  The sweep REDs only the edges whose
+// destination is in the lower half of y (64 MB, held with evict_last) and appends the others
+// as (dst, contribution) records to a spill list (a warp-aggregated append, streamed); a second
+// kernel streams the records and REDs them into the upper half (also 64 MB).  Records beyond
+// the spill capacity are RED'd directly (always correct).
+template <typename A, int U>
+__global__ void __launch_bounds__(TA) k_pr_push_split(const uint64_t *__restrict__ key,
+                                                      const uint32_t *__restrict__ tmask,
+                                                      const uint64_t *__restrict__ head, uint32_t L, uint64_t cap,
+                                                      const A *__restrict__ contrib, A *y, uint32_t rb, uint32_t nr,
+                                                      uint32_t dsplit, uint32_t *__restrict__ sd, A *__restrict__ sc,
+                                                      unsigned long long *scount, uint64_t scap,
+                                                      const uint32_t *__restrict__ done) {
+  if (done && *done) return;
+  const int lane = threadIdx.x & 31;
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
+  const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  const uint64_t w = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32;
+  const uint64_t chunk = (((cap + nwarps - 1) / nwarps) + 32 * U - 1) / (32 * U) * (32 * U);
+  const uint64_t beg = w * chunk, end = min(beg + chunk, cap);
+  if (beg >= end) return;
+  const uint64_t h0 = head[leaf_div(beg, L)];
+  if (h0 == KEY_NONE) return;
+  uint32_t ub = (uint32_t)(h0 >> 32) - rb;
+  A win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
+  uint64_t k[U], kn[U];
+  uint32_t tb[U], tbn[U];
+  auto fetch = [&](uint64_t base, uint64_t *kk, uint32_t *tt) {
+#pragma unroll
+    for (int j = 0; j < U; ++j) {
+      const uint64_t s = base + j * 32 + lane;
+      kk[j] = s < end ? __ldcs(key + s) : KEY_NONE;
+      tt[j] = s < end ? (__ldg(tmask + leaf_div(s, L)) >> leaf_mod(s, L)) & 1u : 1u;
+    }
+  };
+  fetch(beg, k, tb);
+  for (uint64_t base = beg; base < end; base += 32 * U) {
+    if (base + 32 * U < end) fetch(base + 32 * U, kn, tbn);
+#pragma unroll
+    for (int j = 0; j < U; ++j) {
+      const uint32_t dv = (uint32_t)k[j];
+      const bool e = live_key(k[j]) && !tb[j];
+      const uint32_t u = (uint32_t)(k[j] >> 32) - rb;
+      uint32_t pending = __ballot_sync(0xffffffffu, e);
+      while (pending) {
+        const bool mine = (pending >> lane) & 1u;
+        const uint32_t off = mine ? u - ub : 0u;
+        const bool in = mine && off < 32u;
+        const A c = __shfl_sync(0xffffffffu, win, off & 31u);
+        const bool spill = in && dv >= dsplit;
+        const uint32_t sb = __ballot_sync(0xffffffffu, spill);
+        unsigned long long base_s = 0;
+        if (sb && lane == __ffs(sb) - 1) base_s = atomicAdd(scount, (unsigned long long)__popc(sb));
+        base_s = __shfl_sync(0xffffffffu, base_s, sb ? __ffs(sb) - 1 : 0);
+        if (in) {
+          if (spill) {
+            const uint64_t q = base_s + __popc(sb & ((1u << lane) - 1u));
+            if (q < scap) {
+              __stcs(sd + q, dv);
+              __stcs(sc + q, c);
+            } else {
+              red_add_hint(&y[dv], c, pol);
+            }
+          } else {
+            red_add_hint(&y[dv], c, pol);
+          }
+        }
+        pending &= ~__ballot_sync(0xffffffffu, in);
+        if (pending) {
+          ub = __reduce_min_sync(0xffffffffu, ((pending >> lane) & 1u) ? u : 0xFFFFFFFFu);
+          win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
+        }
+      }
+    }
+#pragma unroll
+    for (int j = 0; j < U; ++j) {
+      k[j] = kn[j];
+      tb[j] = tbn[j];
+    }
+  }
+}
+
+template <typename A>
+__global__ void __launch_bounds__(TA) k_pr_spill_apply(const uint32_t *__restrict__ sd, const A *__restrict__ sc,
+                                                       const unsigned long long *scount, uint64_t scap, A *y,
+                                                       const uint32_t *__restrict__ done) {
+  if (done && *done) return;
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
+  const uint64_t n = min((uint64_t)*scount, scap);
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x)
+    red_add_hint(&y[__ldcs(sd + i)], __ldcs(sc + i), pol);
+}
+
+__global__ void k_pr_spill_reset(unsigned long long *scount, const uint32_t *__restrict__ done) {
+  if (done && *done) return;
+  *scount = 0;
+}
+
 // x' = (1-d)/V + d (y + D/V); err += |x'-x|; next contrib / dangling; y := 0
 template <typename T>
 __global__ void k_pr_step(T *__restrict__ x, typename PrAcc<T>::A *__restrict__ y,
@@ -947,6 +1048,12 @@ static int pr_hint() {
   return v;
 }
 
+// GPMA_PR_SPLIT=1: the split push (lower-half REDs in the sweep, upper half through a spill list)
+static bool pr_split() {
+  const char *e = getenv("GPMA_PR_SPLIT");
+  return e && atoi(e) != 0;
+}
+
 static uint32_t pr_passes(uint64_t ybytes) {
   (void)ybytes;
   uint64_t p = 1;
@@ -963,12 +1070,26 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   const uint64_t V = g->V;
   GP_CHECK(g, ensure(g, X.b[1], (V + 1) * sizeof(A), s));
   GP_CHECK(g, ensure(g, X.b[2], (V + 1) * sizeof(A), s));
-  GP_CHECK(g, ensure(g, X.b[3], 4 * sizeof(double) + sizeof(PrLoop), s));
+  GP_CHECK(g, ensure(g, X.b[3], 8 * sizeof(double), s));   // acc[0..3], PrLoop at acc + 4, spill count at acc + 6
   const uint32_t *deg = g->deg;
   A *contrib = (A *)X.b[1].p, *y = (A *)X.b[2].p;
   double *acc = (double *)X.b[3].p;   // [0],[1] dangling ping-pong, [2] error, then the loop state
   PrLoop *lp = (PrLoop *)(acc + 4);
   const uint32_t passes = pr_passes(V * sizeof(A));
+  // split push: a spill list for half of the slots (records past it are RED'd directly)
+  const bool split = pr_split() && passes == 1;
+  uint32_t *sd = nullptr;
+  A *sc = nullptr;
+  unsigned long long *scount = nullptr;
+  uint64_t scap = 0;
+  if (split) {
+    scap = g->cap / 2;
+    GP_CHECK(g, ensure(g, X.stage[0], scap * 4 + 16, s));
+    GP_CHECK(g, ensure(g, X.stage[1], scap * sizeof(A) + 16, s));
+    sd = (uint32_t *)X.stage[0].p;
+    sc = (A *)X.stage[1].p;
+    scount = (unsigned long long *)(acc + 6);
+  }
   GP_CHECK(g, fill_zero(g, acc, 4 * sizeof(double) + sizeof(PrLoop), s));
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
   // Iterations are queued in batches (2 first: a warm start rarely stops after one, then 1
@@ -982,11 +1103,18 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
     const int batch = tol <= 0.0 ? max_iter - queued : std::min(queued == 0 ? 2 : 1, max_iter - queued);
     for (int b = 0; b < batch; ++b, ++queued) {
       GP_LAUNCH(g, k_pr_iter_begin, 1, 32, 0, s, acc, cur ^ 1, lp);
-      // destination passes: random REDs run ~3x faster while their target fits in L2
-      for (uint32_t q = 0; q < passes; ++q)
-        GP_LAUNCH(g, (k_pr_push_win<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
-                  g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes),
-                  pr_hint(), &lp->done);
+      if (split) {
+        GP_LAUNCH(g, k_pr_spill_reset, 1, 1, 0, s, scount, &lp->done);
+        GP_LAUNCH(g, (k_pr_push_split<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L, g->cap,
+                  contrib, y, 0u, g->nr, (uint32_t)(V / 2), sd, sc, scount, scap, &lp->done);
+        GP_LAUNCH(g, k_pr_spill_apply<A>, grid_cap(), TA, 0, s, sd, sc, scount, scap, y, &lp->done);
+      } else {
+        // destination passes: random REDs run ~3x faster while their target fits in L2
+        for (uint32_t q = 0; q < passes; ++q)
+          GP_LAUNCH(g, (k_pr_push_win<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L,
+                    g->cap, contrib, y, 0u, g->nr, (uint32_t)(V * q / passes), (uint32_t)(V * (q + 1) / passes),
+                    pr_hint(), &lp->done);
+      }
       GP_LAUNCH(g, k_pr_step<T>, grid_for(V), TA, 0, s, x, y, deg, contrib, (uint32_t)V, d, acc + cur,
                 acc + (cur ^ 1), acc + 2, &lp->done);
       GP_LAUNCH(g, k_pr_iter_end, 1, 32, 0, s, acc, tol, lp);

@@ -368,3 +368,33 @@ def test_gpma_lock_hot_rows_and_doubling(seed):
         o.insert(ks, vs)
         assert_same_layout(g, o, what=f"gpma hot seed {seed} step {step}")
     assert g.gpma_stats()["resizes"] == o.stats()["resizes"] > 0
+
+
+@pytest.mark.parametrize("split", ["0", "1"])
+def test_pagerank_push_strategies(split, monkeypatch):
+    """The PageRank push with and without the split (GPMA_PR_SPLIT: lower-half destinations RED'd in
+    the sweep, upper half through a spill list) against the oracle, fp64 and fp32, fixed K and the
+    tolerance mode (same stopping iteration)."""
+    monkeypatch.setenv("GPMA_PR_SPLIT", split)
+    from gpma_gen.streams import StreamConfig
+    cfg = StreamConfig("rmat-s16", "rmat", 1 << 16, 1 << 20, 1 << 19, 1 << 15, 0x5EED + 3, scale=16)
+    sw = config_stream(cfg, device=DEV)
+    sw.keys, sw.vals = sw.keys.cpu(), sw.vals.cpu()
+    V = 1 << 16
+    k0, v0 = sw.initial()
+    g = Gpma.gpma_create(V, k0.to(DEV), v0.to(DEV))
+    o = O.Oracle(V, k0, v0)
+    dk, ik, iv = sw.slide(0)
+    g.delete(dk.to(DEV))
+    g.insert(ik.to(DEV), iv.to(DEV))
+    o.delete(dk)
+    o.insert(ik, iv)
+    xg, _ = gpu_pr(g, tol=0.0, max_iter=7)
+    xo, _ = o.pagerank(tol=0.0, max_iter=7)
+    assert_pr_close(xg, xo, what=f"split={split} fp64")
+    x32, _ = gpu_pr(g, tol=0.0, max_iter=7, dtype=torch.float32)
+    assert_pr_close(x32, xo, fp64=False, what=f"split={split} fp32")
+    xg, itg = gpu_pr(g, xg, tol=1e-3, max_iter=100)
+    xo2, ito = o.pagerank(x=xo, tol=1e-3, max_iter=100)
+    assert itg == ito
+    assert_pr_close(xg, xo2, what=f"split={split} tolerance mode")
