@@ -158,6 +158,7 @@ void free_handle(gpma *g) {
     DevBuf *xb[] = {&x.b[0], &x.b[1], &x.b[2], &x.b[3], &x.misc, &x.lpre, &x.scan, &x.stage[0], &x.stage[1]};
     for (DevBuf *b : xb) gp::release(g, *b, s);
   }
+  gp::spare_release(g, s);
   gp::dev_free(g, g->key, s);
   gp::dev_free(g, g->val, s);
   gp::dev_free(g, g->cnt, s);

@@ -104,6 +104,14 @@ struct gpma {
   uint32_t rho0 = 800, rhoh = 4000, tau0 = 9200, tauh = 8000, init_bp = 6000;
   std::vector<uint64_t> tmin, tmax;
 
+  struct SpareStore {              // the previous capacity's arrays, kept across a resize
+    uint64_t cap = 0;
+    uint64_t *key = nullptr;
+    uint32_t *val = nullptr;
+    uint32_t *cnt = nullptr;
+    uint64_t *head = nullptr;
+  } spare;
+
   // store (HBM-resident)
   uint64_t *key = nullptr;        // [cap]
   uint32_t *val = nullptr;        // [cap]
@@ -273,6 +281,7 @@ gpma_status build_from_sorted(gpma *g, const uint64_t *sk, const uint32_t *sv, u
                               cudaStream_t s);
 gpma_status load_raw(gpma *g, const uint64_t *keys, const uint32_t *vals, cudaStream_t s);
 gpma_status recompute_heads(gpma *g, cudaStream_t s);
+void spare_release(gpma *g, cudaStream_t s);
 gpma_status count_slots(gpma *g, uint64_t *live_edges, uint64_t *tombs, cudaStream_t s);
 gpma_status recompute_degrees(gpma *g, cudaStream_t s);   // analytics.cu
 inline uint32_t *tmask_of(gpma *g) { return g->cnt + g->cap / g->L; }

@@ -58,11 +58,22 @@ void pool_attach(gpma *g) {
   g->pool_attached = true;
 }
 
+// When the device's last handle goes, the pool is trimmed down to GPMA_POOL_KEEP_MB (default: a
+// quarter of the device's memory): a later store of the process (e.g. the next pass of a
+// benchmark, a re-created graph) reuses mapped blocks instead of mapping GBs again -- mapping is
+// what made round-1 resizing steps vary from 16 ms to 1.1 s -- while the rest goes back to the
+// driver for a co-resident allocator (PyTorch's).
 void pool_detach(gpma *g) {
   if (!g->pool_attached) return;
   std::lock_guard<std::mutex> lk(g_pool_mu);
   DevPool &P = g_pools[g->device & 63];
-  if (--P.handles == 0 && P.pool) cudaMemPoolTrimTo(P.pool, 0);   // every block is free by now
+  if (--P.handles == 0 && P.pool) {
+    size_t keep = 0, fr = 0, tot = 0;
+    if (const char *e = getenv("GPMA_POOL_KEEP_MB")) keep = (size_t)atoll(e) << 20;
+    else if (cudaMemGetInfo(&fr, &tot) == cudaSuccess) keep = tot / 4;
+    cudaGetLastError();
+    cudaMemPoolTrimTo(P.pool, keep);                    // every block is free by now
+  }
   g->pool_attached = false;
 }
 

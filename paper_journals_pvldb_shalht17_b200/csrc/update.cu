@@ -2646,20 +2646,64 @@ gpma_status count_slots(gpma *g, uint64_t *live_edges, uint64_t *tombs, cudaStre
   return GPMA_OK;
 }
 
+// GPMA_SPARE=0 frees the old store arrays at a resize instead of keeping them as a spare set
+static bool spare_on() {
+  const char *e = getenv("GPMA_SPARE");
+  return !e || atoi(e) != 0;
+}
+
 static void set_geometry(gpma *g, uint64_t cap) {
   g->cap = cap;
   g->h = ilog2(cap / g->L);
   level_bounds(g->L, g->h, g->rho0, g->rhoh, g->tau0, g->tauh, g->tmin, g->tmax);
 }
 
+// The store arrays of the previous capacity are kept as a spare set across a resize, so the
+// dual resize (a halving after a doubling, a doubling after a halving) takes them back instead
+// of allocating -- and mapping -- GBs (round-1 resizing steps varied 16 ms - 1.1 s).
+static void spare_stash(gpma *g, uint64_t cap, uint64_t *k, uint32_t *v, uint32_t *c, uint64_t *hd, cudaStream_t s) {
+  if (g->spare.key) {
+    dev_free(g, g->spare.key, s);
+    dev_free(g, g->spare.val, s);
+    dev_free(g, g->spare.cnt, s);
+    dev_free(g, g->spare.head, s);
+  }
+  g->spare.cap = cap;
+  g->spare.key = k;
+  g->spare.val = v;
+  g->spare.cnt = c;
+  g->spare.head = hd;
+}
+
+void spare_release(gpma *g, cudaStream_t s) { spare_stash(g, 0, nullptr, nullptr, nullptr, nullptr, s); }
+
 static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v, uint32_t **c,
                                uint64_t **hd, cudaStream_t s) {
   uint64_t nl = cap / g->L;
+  if (g->spare.key && g->spare.cap == cap && spare_on()) {
+    *k = g->spare.key;
+    *v = g->spare.val;
+    *c = g->spare.cnt;
+    *hd = g->spare.head;
+    g->spare = gpma::SpareStore{};
+    return GPMA_OK;
+  }
   *k = nullptr; *v = nullptr; *c = nullptr; *hd = nullptr;
   cudaError_t e1 = dev_alloc(g, (void **)k, cap * 8, s);
   cudaError_t e2 = dev_alloc(g, (void **)v, cap * 4, s);
   cudaError_t e3 = dev_alloc(g, (void **)c, nl * 12, s);  // live counts, tombstone masks, guards
   cudaError_t e4 = dev_alloc(g, (void **)hd, nl * 8, s);
+  if ((e1 || e2 || e3 || e4) && g->spare.key) {          // out of memory: give the spare set back first
+    dev_free(g, *k, s);
+    dev_free(g, *v, s);
+    dev_free(g, *c, s);
+    dev_free(g, *hd, s);
+    spare_release(g, s);
+    e1 = dev_alloc(g, (void **)k, cap * 8, s);
+    e2 = dev_alloc(g, (void **)v, cap * 4, s);
+    e3 = dev_alloc(g, (void **)c, nl * 12, s);
+    e4 = dev_alloc(g, (void **)hd, nl * 8, s);
+  }
   if (e1 || e2 || e3 || e4) {
     cudaGetLastError();
     dev_free(g, *k, s);
@@ -3044,10 +3088,14 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   LevelOut lo{};
   if ((st = level_step(g, a, cur, &lo, dirty_base, s, true, cap, nk, nv, ncnt))) return st;
   if (cap != g->cap) {
-    dev_free(g, g->key, s);
-    dev_free(g, g->val, s);
-    dev_free(g, g->cnt, s);
-    dev_free(g, g->head, s);
+    if (spare_on()) {
+      spare_stash(g, g->cap, g->key, g->val, g->cnt, g->head, s);
+    } else {
+      dev_free(g, g->key, s);
+      dev_free(g, g->val, s);
+      dev_free(g, g->cnt, s);
+      dev_free(g, g->head, s);
+    }
     g->key = nk;
     g->val = nv;
     g->cnt = ncnt;
@@ -3265,10 +3313,14 @@ static gpma_status double_root(gpma *g, cudaStream_t s) {
   if ((st = alloc_store(g, cap2, &nk, &nv, &ncnt, &nhead, s))) return st;
   GP_LAUNCH(g, k_layout_even, grid_for(cap2 / 4), TB, 0, s, (const uint64_t *)g->b_wk.p, (const uint32_t *)g->b_wv.p,
             N, nk, nv, ncnt, g->row_offset, g->L, cap2 / g->L, g->rb);
-  dev_free(g, g->key, s);
-  dev_free(g, g->val, s);
-  dev_free(g, g->cnt, s);
-  dev_free(g, g->head, s);
+  if (spare_on()) {
+    spare_stash(g, g->cap, g->key, g->val, g->cnt, g->head, s);
+  } else {
+    dev_free(g, g->key, s);
+    dev_free(g, g->val, s);
+    dev_free(g, g->cnt, s);
+    dev_free(g, g->head, s);
+  }
   g->key = nk;
   g->val = nv;
   g->cnt = ncnt;
