@@ -886,7 +886,7 @@ __global__ void __launch_bounds__(TA) k_pr_push_split(const uint64_t *__restrict
                                                       const uint64_t *__restrict__ head, uint32_t L, uint64_t cap,
                                                       const A *__restrict__ contrib, A *y, uint32_t rb, uint32_t nr,
                                                       uint32_t dsplit, uint32_t *__restrict__ sd, A *__restrict__ sc,
-                                                      unsigned long long *scount, uint64_t scap,
+                                                      unsigned long long *__restrict__ scount,
                                                       const uint32_t *__restrict__ done) {
   if (done && *done) return;
   const int lane = threadIdx.x & 31;
@@ -896,9 +896,16 @@ __global__ void __launch_bounds__(TA) k_pr_push_split(const uint64_t *__restrict
   const uint64_t w = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32;
   const uint64_t chunk = (((cap + nwarps - 1) / nwarps) + 32 * U - 1) / (32 * U) * (32 * U);
   const uint64_t beg = w * chunk, end = min(beg + chunk, cap);
-  if (beg >= end) return;
+  if (beg >= end) {
+    if (lane == 0) scount[w] = 0;
+    return;
+  }
+  uint64_t nsp = 0;                                      // records spilled by this warp (<= its slots)
   const uint64_t h0 = head[leaf_div(beg, L)];
-  if (h0 == KEY_NONE) return;
+  if (h0 == KEY_NONE) {
+    if (lane == 0) scount[w] = 0;
+    return;
+  }
   uint32_t ub = (uint32_t)(h0 >> 32) - rb;
   A win = (ub + lane < nr) ? __ldcs(contrib + ub + lane) : A(0);
   uint64_t k[U], kn[U];
@@ -927,22 +934,16 @@ __global__ void __launch_bounds__(TA) k_pr_push_split(const uint64_t *__restrict
         const A c = __shfl_sync(0xffffffffu, win, off & 31u);
         const bool spill = in && dv >= dsplit;
         const uint32_t sb = __ballot_sync(0xffffffffu, spill);
-        unsigned long long base_s = 0;
-        if (sb && lane == __ffs(sb) - 1) base_s = atomicAdd(scount, (unsigned long long)__popc(sb));
-        base_s = __shfl_sync(0xffffffffu, base_s, sb ? __ffs(sb) - 1 : 0);
         if (in) {
-          if (spill) {
-            const uint64_t q = base_s + __popc(sb & ((1u << lane) - 1u));
-            if (q < scap) {
-              __stcs(sd + q, dv);
-              __stcs(sc + q, c);
-            } else {
-              red_add_hint(&y[dv], c, pol);
-            }
+          if (spill) {                                   // the warp's private spill run (no atomics)
+            const uint64_t q = beg + nsp + __popc(sb & ((1u << lane) - 1u));
+            __stcs(sd + q, dv);
+            __stcs(sc + q, c);
           } else {
             red_add_hint(&y[dv], c, pol);
           }
         }
+        nsp += __popc(sb);
         pending &= ~__ballot_sync(0xffffffffu, in);
         if (pending) {
           ub = __reduce_min_sync(0xffffffffu, ((pending >> lane) & 1u) ? u : 0xFFFFFFFFu);
@@ -956,23 +957,24 @@ __global__ void __launch_bounds__(TA) k_pr_push_split(const uint64_t *__restrict
       tb[j] = tbn[j];
     }
   }
+  if (lane == 0) scount[w] = nsp;
 }
 
+// the spill runs: warp w of the push wrote scount[w] records at the start of its slot chunk
 template <typename A>
 __global__ void __launch_bounds__(TA) k_pr_spill_apply(const uint32_t *__restrict__ sd, const A *__restrict__ sc,
-                                                       const unsigned long long *scount, uint64_t scap, A *y,
-                                                       const uint32_t *__restrict__ done) {
+                                                       const unsigned long long *__restrict__ scount, uint64_t cap,
+                                                       uint64_t nwarps_push, A *y, const uint32_t *__restrict__ done) {
   if (done && *done) return;
   uint64_t pol;
   asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
-  const uint64_t n = min((uint64_t)*scount, scap);
-  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x)
-    red_add_hint(&y[__ldcs(sd + i)], __ldcs(sc + i), pol);
-}
-
-__global__ void k_pr_spill_reset(unsigned long long *scount, const uint32_t *__restrict__ done) {
-  if (done && *done) return;
-  *scount = 0;
+  const int lane = threadIdx.x & 31;
+  const uint64_t chunk = (((cap + nwarps_push - 1) / nwarps_push) + 32 * 4 - 1) / (32 * 4) * (32 * 4);
+  const uint64_t nwarps = (uint64_t)gridDim.x * (blockDim.x / 32);
+  for (uint64_t w = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32; w < nwarps_push; w += nwarps) {
+    const uint64_t n = scount[w], base = w * chunk;
+    for (uint64_t i = lane; i < n; i += 32) red_add_hint(&y[__ldcs(sd + base + i)], __ldcs(sc + base + i), pol);
+  }
 }
 
 // x' = (1-d)/V + d (y + D/V); err += |x'-x|; next contrib / dangling; y := 0
@@ -1082,13 +1084,14 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
   A *sc = nullptr;
   unsigned long long *scount = nullptr;
   uint64_t scap = 0;
-  if (split) {
-    scap = g->cap / 2;
+  if (split) {                                     // a private run per push warp: cap records
+    scap = g->cap + 32 * 4 * (uint64_t)SWEEP_BLOCKS * (TA / 32);
     GP_CHECK(g, ensure(g, X.stage[0], scap * 4 + 16, s));
     GP_CHECK(g, ensure(g, X.stage[1], scap * sizeof(A) + 16, s));
+    GP_CHECK(g, ensure(g, X.misc, (uint64_t)SWEEP_BLOCKS * (TA / 32) * 8, s));
     sd = (uint32_t *)X.stage[0].p;
     sc = (A *)X.stage[1].p;
-    scount = (unsigned long long *)(acc + 6);
+    scount = (unsigned long long *)X.misc.p;
   }
   GP_CHECK(g, fill_zero(g, acc, 4 * sizeof(double) + sizeof(PrLoop), s));
   GP_LAUNCH(g, k_pr_prep<T>, grid_for(V), TA, 0, s, x, deg, contrib, y, (uint32_t)V, warm ? 0 : 1, acc);
@@ -1104,10 +1107,10 @@ static gpma_status pagerank_t(gpma *g, T *x, int warm, T d, double tol, int max_
     for (int b = 0; b < batch; ++b, ++queued) {
       GP_LAUNCH(g, k_pr_iter_begin, 1, 32, 0, s, acc, cur ^ 1, lp);
       if (split) {
-        GP_LAUNCH(g, k_pr_spill_reset, 1, 1, 0, s, scount, &lp->done);
         GP_LAUNCH(g, (k_pr_push_split<A, 4>), SWEEP_BLOCKS, TA, 0, s, g->key, tmask_of(g), g->head, g->L, g->cap,
-                  contrib, y, 0u, g->nr, (uint32_t)(V / 2), sd, sc, scount, scap, &lp->done);
-        GP_LAUNCH(g, k_pr_spill_apply<A>, grid_cap(), TA, 0, s, sd, sc, scount, scap, y, &lp->done);
+                  contrib, y, 0u, g->nr, (uint32_t)(V / 2), sd, sc, scount, &lp->done);
+        GP_LAUNCH(g, k_pr_spill_apply<A>, grid_cap(), TA, 0, s, sd, sc, scount, g->cap,
+                  (uint64_t)SWEEP_BLOCKS * (TA / 32), y, &lp->done);
       } else {
         // destination passes: random REDs run ~3x faster while their target fits in L2
         for (uint32_t q = 0; q < passes; ++q)

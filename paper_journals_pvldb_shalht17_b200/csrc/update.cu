@@ -3593,12 +3593,16 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
 }
 
 // GPMA_SMALL=0 disables the one-kernel small-batch path (read per call)
+// GPMA_SMALL=0 disables the one-kernel small-batch path; GPMA_SMALL=<n> sets the largest insert
+// batch it takes (default 256: one round of leaf rows -- beyond it the single CTA serialises what
+// the multi-kernel path spreads over the GPU; deletes up to 8x that).  Read per call.
 static bool small_batch_path(gpma *g, uint64_t n, int op, int path) {
-  const char *e = getenv("GPMA_SMALL");
-  if (e && atoi(e) == 0) return false;
-  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) return n <= (uint64_t)SB_DEL_MAX;
+  uint64_t lim = SB_ROWS;
+  if (const char *e = getenv("GPMA_SMALL")) lim = std::min<uint64_t>((uint64_t)atoll(e), SB_MAX);
+  if (lim == 0) return false;
+  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) return n <= std::min<uint64_t>(8 * lim, SB_DEL_MAX);
   if (path == PATH_INS_LEAF || path == PATH_INS_FUSED)
-    return n <= (uint64_t)SB_MAX && (g->L == 4 || g->L == 8 || g->L == 16);
+    return n <= lim && (g->L == 4 || g->L == 8 || g->L == 16);
   return false;
 }
 

@@ -145,14 +145,15 @@ def test_config0_sliding_window_graph_replay(seed):
 
 @pytest.mark.parametrize("knob", ["GPMA_DEL_SORT=1", "GPMA_INS_FUSED=0", "GPMA_INS_LEAFSORT=0",
                                   "GPMA_INS_LEAFSORT=0,GPMA_INS_THREAD=0", "GPMA_LVL_COOP=0", "GPMA_ILP=1",
-                                  "GPMA_ILP=4", "GPMA_SMALL=0", "GPMA_SMALL=0,GPMA_DEL_SORT=1"])
+                                  "GPMA_ILP=4", "GPMA_SMALL=2048", "GPMA_SMALL=0,GPMA_DEL_SORT=1"])
 @pytest.mark.parametrize("seed", range(3))
 def test_config0_alternative_paths(seed, knob, monkeypatch):
     """The strategy switches give the same layouts as the defaults (configs[0] batches are 1024 keys:
-    by default the one-kernel small-batch path; GPMA_SMALL=0 sends them through the large-batch
-    kernels -- leaf-keyed insert, interleaved lazy delete -- and the other knobs through the
-    alternatives: sorted lazy delete, separate pre-pass + k_level0, key-sorted fused insert by a
-    thread or a sub-warp per leaf, the host-driven level loop, 1- or 4-way probe interleaving)."""
+    by default the large-batch kernels -- leaf-keyed insert, interleaved lazy delete; GPMA_SMALL=2048
+    sends them through the one-kernel small-batch path (4 rounds of leaf rows) -- and the other
+    knobs through the alternatives: sorted lazy delete, separate pre-pass + k_level0, key-sorted
+    fused insert by a thread or a sub-warp per leaf, the host-driven level loop, 1- or 4-way probe
+    interleaving)."""
     for kv in knob.split(","):
         k, v = kv.split("=")
         monkeypatch.setenv(k, v)
