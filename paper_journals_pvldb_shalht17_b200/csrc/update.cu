@@ -3738,21 +3738,44 @@ static gpma_status run_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
 // flagged the batch, so the common insert path (sort -> pre-pass -> fused level 0) needs a
 // single host round trip; the generic levels >= 1 and the resize follow only when level 0
 // leaves updates pending.
+static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int path,
+                                       const Sorted &srt, cudaStream_t s);
+
+static bool is_device_ptr(const void *p) {
+  if (!p) return false;
+  cudaPointerAttributes a{};
+  if (cudaPointerGetAttributes(&a, p) != cudaSuccess) {
+    cudaGetLastError();
+    return false;
+  }
+  return a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged;
+}
+
 gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, int op,
                          cudaStream_t s) {
   gpma_status st;
   g->last = gpma_stats_t{};
   g->trace.clear();
   if (n == 0) return GPMA_OK;
+  int path = prefix_path(g, op);
+  Sorted srt;
+  if (small_batch_path(g, n, op, path) && is_device_ptr(keys) && (op != GPMA_INSERT || is_device_ptr(vals))) {
+    // the one-kernel small batch only reads the batch: no staging copy of a device batch
+    if ((st = run_small(g, const_cast<uint64_t *>(keys), const_cast<uint32_t *>(vals), n, op, s))) return st;
+    path = path == PATH_INS_LEAF || path == PATH_INS_FUSED ? PATH_INS_SMALL : path;
+    GP_CHECK(g, cudaStreamSynchronize(s));
+    if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) {
+      g->last.last_unique = n;
+      return status_of(g);
+    }
+    return update_after_prefix(g, keys, vals, n, op, path, srt, s);
+  }
   GP_CHECK(g, ensure(g, g->b_stage[0], n * 8, s));
   GP_CHECK(g, ensure(g, g->b_stage[1], n * 4, s));
   uint64_t *ik = (uint64_t *)g->b_stage[0].p;
   uint32_t *iv = (uint32_t *)g->b_stage[1].p;
   GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));
   if (op == GPMA_INSERT) GP_CHECK(g, stage_in(g, iv, vals, n * 4, s));
-  const uint64_t nl = g->cap / g->L;
-  int path = prefix_path(g, op);
-  Sorted srt;
   if (small_batch_path(g, n, op, path)) {
     if ((st = run_small(g, ik, iv, n, op, s))) return st;
     path = path == PATH_INS_LEAF || path == PATH_INS_FUSED ? PATH_INS_SMALL : path;
@@ -3764,6 +3787,15 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
     g->last.last_unique = n;   // (lazy deletes are idempotent; the sorted path marks each key once)
     return status_of(g);
   }
+  return update_after_prefix(g, ik, iv, n, op, path, srt, s);
+}
+
+// After the prefix's host round trip: the pending list of level 1 (if any), the level loop, the
+// root resize, the head fix-up.  ik / iv: the batch the prefix read (staged or the caller's).
+static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int path,
+                                       const Sorted &srt, cudaStream_t s) {
+  gpma_status st;
+  const uint64_t nl = g->cap / g->L;
   uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
   const bool lock = op == GPMA_INSERT && g->algorithm == 1;   // GPMA (Alg. 1) instead of GPMA+
   const bool fused = !g->trace_on && !lock;
