@@ -56,6 +56,8 @@ def parse():
     ap.add_argument("--force-dist", action="store_true", help="use the sharded path even at N=1 (testing)")
     ap.add_argument("--no-sweep", action="store_true", help="skip the configs[1] batch-size sweep")
     ap.add_argument("--no-resize", action="store_true", help="skip the configs[3] grow/shrink resize stress")
+    ap.add_argument("--log-jsonl", default="", help="per-slide JSONL log of the timed steps (phase ms, PR "
+                    "iterations, levels climbed, slots rewritten, resizes) -- written after the timed region")
     ap.add_argument("--concurrent-analytics", action="store_true",
                     help="run BFS/CC/PR/export side by side on 4 streams (fanout.py) instead of one "
                          "after another (the default: per-phase breakdown, uncontended roofline)")
@@ -213,6 +215,7 @@ def run_gpma(args, rank, world, lrank):
         st0 = g.gpma_stats()
         evs = []
         pr_iters = []
+        slide_log = []
 
         # priorities: the latency-bound BFS and CC levels jump the queue of the sweep kernels
         fan = AnalyticsFanout(dev, timing=True, priorities=[0, -1, -2, 0]) if args.concurrent_analytics else None
@@ -230,6 +233,13 @@ def run_gpma(args, rank, world, lrank):
             e[1].record(s)
             g.gpma_update_batch(ikk, ivv, 0, stream=s)
             e[2].record(s)
+            if args.log_jsonl:                         # host-side counters only (no device work)
+                st_h = g.gpma_stats_host()
+                slide_log.append({"slide": i, "top_level": st_h["last_top_level"],
+                                  "slots_rewritten": st_h["last_slots_rewritten"],
+                                  "windows_rewritten": st_h["last_windows_rewritten"],
+                                  "pending_after_prepass": st_h["last_pending"], "resized": st_h["last_resized"],
+                                  "capacity": st_h["capacity"]})
             if fan is None:                    # serial: one stream, phase by phase
                 g.gpma_bfs(root, lv, stream=s)
                 e[3].record(s)
@@ -302,6 +312,12 @@ def run_gpma(args, rank, world, lrank):
                          "pagerank": per[0], "cc": per[1], "bfs": per[2], "export_csr": per[3],
                          "analytics": "concurrent: 4 streams / 4 host threads (per-analytic times overlap)"}
         iters_timed = list(pr_iters)
+        if args.log_jsonl and fan is None:
+            with open(args.log_jsonl, "w") as f:
+                for rec, ph, it_ in zip(slide_log[-len(evs):], phase.tolist(), iters_timed):
+                    rec.update({"delete_ms": ph[0], "insert_ms": ph[1], "bfs_ms": ph[2], "cc_ms": ph[3],
+                                "pagerank_ms": ph[4], "export_ms": ph[5], "pr_iters": it_})
+                    f.write(json.dumps(rec) + "\n")
         st = g.gpma_stats()
         cap = st["capacity"]
         slide_ms = phase[:, 0] + phase[:, 1]

@@ -174,6 +174,9 @@ gpma_status gpma_export_csr(gpma_t *g, uint64_t *row_ptr, uint32_t *col, uint32_
                             uint64_t nnz_capacity, uint64_t *nnz_out, gpma_stream_t stream);
 
 gpma_status gpma_stats(gpma_t *g, gpma_stats_t *out);
+/* The same without any device work (no synchronisation): live_edges and tombstones are set to
+ * UINT64_MAX (not counted); everything else as gpma_stats.  For per-batch logging. */
+gpma_status gpma_stats_host(const gpma_t *g, gpma_stats_t *out);
 
 /* Parity hooks.  Raw layout: keys u64[capacity] (0xFFFF..FF = empty), vals
  * u32[capacity] (0 on empty slots); row_offset u64[V+1] (R8); leaf_live u32[cap/L]

@@ -335,6 +335,7 @@ gpma_status gpma_destroy(gpma_t *g) {
 
 gpma_status gpma_update_batch(gpma_t *g, const uint64_t *keys, const uint32_t *vals, uint64_t n, gpma_op op,
                               gpma_stream_t stream) {
+  gp::Nvtx nvtx_("gpma_update_batch");
   gpma_status st = begin(g);
   if (st) return st;
   if (op != GPMA_INSERT && op != GPMA_DELETE) return GPMA_ERR_INVALID_ARG;
@@ -354,6 +355,7 @@ gpma_status gpma_update_batch(gpma_t *g, const uint64_t *keys, const uint32_t *v
 }
 
 gpma_status gpma_bfs(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t stream) {
+  gp::Nvtx nvtx_("gpma_bfs");
   gpma_status st = begin(g);
   if (st) return st;
   if (!levels || root >= g->V) return GPMA_ERR_INVALID_ARG;
@@ -368,6 +370,7 @@ gpma_status gpma_bfs(gpma_t *g, uint32_t root, int32_t *levels, gpma_stream_t st
 }
 
 gpma_status gpma_cc(gpma_t *g, uint32_t *labels, gpma_stream_t stream) {
+  gp::Nvtx nvtx_("gpma_cc");
   gpma_status st = begin(g);
   if (st) return st;
   if (!labels) return GPMA_ERR_INVALID_ARG;
@@ -383,6 +386,7 @@ gpma_status gpma_cc(gpma_t *g, uint32_t *labels, gpma_stream_t stream) {
 
 gpma_status gpma_pagerank(gpma_t *g, double *rank, int warm_start, double damping, double tol_l1, int max_iter,
                           int *iters_out, gpma_stream_t stream) {
+  gp::Nvtx nvtx_("gpma_pagerank");
   gpma_status st = begin(g);
   if (st) return st;
   if (!rank || max_iter < 0 || !(damping >= 0.0 && damping <= 1.0) || !(tol_l1 >= 0.0)) return GPMA_ERR_INVALID_ARG;
@@ -400,6 +404,7 @@ gpma_status gpma_pagerank(gpma_t *g, double *rank, int warm_start, double dampin
 
 gpma_status gpma_pagerank_f32(gpma_t *g, float *rank, int warm_start, float damping, float tol_l1, int max_iter,
                               int *iters_out, gpma_stream_t stream) {
+  gp::Nvtx nvtx_("gpma_pagerank_f32");
   gpma_status st = begin(g);
   if (st) return st;
   if (g->comm) return GPMA_ERR_INVALID_ARG;
@@ -417,6 +422,7 @@ gpma_status gpma_pagerank_f32(gpma_t *g, float *rank, int warm_start, float damp
 
 gpma_status gpma_export_csr(gpma_t *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val, uint64_t nnz_capacity,
                             uint64_t *nnz_out, gpma_stream_t stream) {
+  gp::Nvtx nvtx_("gpma_export_csr");
   gpma_status st = begin(g);
   if (st) return st;
   if (col && (!row_ptr || !val)) return GPMA_ERR_INVALID_ARG;
@@ -462,6 +468,25 @@ gpma_status gpma_stats(gpma_t *g, gpma_stats_t *out) {
   out->total_windows_rewritten = g->tot[4];
   st = gp::count_slots(g, &out->live_edges, &out->tombstones, g->st);
   return end(g, st);
+}
+
+gpma_status gpma_stats_host(const gpma_t *g, gpma_stats_t *out) {
+  if (!g || !out) return GPMA_ERR_INVALID_ARG;
+  *out = g->last;
+  out->num_vertices = g->V;
+  out->leaf_slots = g->L;
+  out->capacity = g->cap;
+  out->height = g->h;
+  out->delete_mode = g->mode;
+  out->resizes = g->resizes;
+  out->total_batches = g->tot[0];
+  out->total_insert_keys = g->tot[1];
+  out->total_delete_keys = g->tot[2];
+  out->total_slots_rewritten = g->tot[3];
+  out->total_windows_rewritten = g->tot[4];
+  out->live_edges = ~0ull;
+  out->tombstones = ~0ull;
+  return GPMA_OK;
 }
 
 gpma_status gpma_debug_dump(gpma_t *g, uint64_t *keys, uint32_t *vals, uint64_t *row_offset, uint32_t *leaf_live,

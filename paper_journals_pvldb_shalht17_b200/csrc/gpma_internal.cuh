@@ -10,9 +10,18 @@
 #include <string>
 #include <vector>
 
+#include <nvtx3/nvToolsExt.h>
+
 #include "../../include/gpma.h"
 
 namespace gp {
+
+// NVTX range of a phase (nsys / ncu timelines: every C-ABI call and the phases of an update
+// batch show up by name; header-only NVTX3, inert unless a tool is attached)
+struct Nvtx {
+  explicit Nvtx(const char *name) { nvtxRangePushA(name); }
+  ~Nvtx() { nvtxRangePop(); }
+};
 
 constexpr uint64_t KEY_NONE = ~0ull;          // R2 empty slot
 constexpr uint32_t VAL_TOMB = 0xFFFFFFFFu;    // R12 lazy-delete mark

@@ -3051,6 +3051,7 @@ static Lvl make_lvl(gpma *g, int cur, uint64_t p, uint32_t lvl, int op) {
 // insertions fit max_h of the new capacity; halve (strict deletes) while below min_h
 // and cap > 2L.  Everything is laid out evenly over the new array.
 static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, uint64_t *dirty_base) {
+  Nvtx nvtx_("update: root resize");
   gpma_status st;
   uint64_t nl = g->cap / g->L;
   if ((st = zero_ctrl(g, s))) return st;
@@ -3759,6 +3760,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   if (n == 0) return GPMA_OK;
   int path = prefix_path(g, op);
   Sorted srt;
+  Nvtx nvtx_(op == GPMA_INSERT ? "update: insert prefix" : "update: delete prefix");
   if (small_batch_path(g, n, op, path) && is_device_ptr(keys) && (op != GPMA_INSERT || is_device_ptr(vals))) {
     // the one-kernel small batch only reads the batch: no staging copy of a device batch
     if ((st = run_small(g, const_cast<uint64_t *>(keys), const_cast<uint32_t *>(vals), n, op, s))) return st;
@@ -3876,8 +3878,10 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     lvl = 1;
   }
   if (p > 0 && lvl >= 1 && lvl <= g->h && !g->trace_on && coop_eligible(g, p, lvl)) {
+    Nvtx nv("update: device level loop");
     if ((st = coop_levels(g, cur, p, lvl, &dirty_base, op, s))) return st;
   }
+  Nvtx nvtx_levels("update: host level loop");
   for (; lvl <= g->h && p > 0; ++lvl) {
     Lvl a = make_lvl(g, cur, p, lvl, op);
     LevelOut lo{};

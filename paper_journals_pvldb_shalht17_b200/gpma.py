@@ -94,6 +94,7 @@ def lib() -> C.CDLL:
             "gpma_pagerank_f32": (st, [P, P, i32, C.c_float, C.c_float, i32, P, P]),
             "gpma_export_csr": (st, [P, P, P, P, u64, P, P]),
             "gpma_stats": (st, [P, P]),
+            "gpma_stats_host": (st, [P, P]),
             "gpma_debug_dump": (st, [P, P, P, P, P, P, P]),
             "gpma_debug_set_trace": (st, [P, i32]),
             "gpma_debug_dump_aux": (st, [P, P, P, P, P]),
@@ -135,7 +136,7 @@ EXPORTS = ["gpma_config_default", "gpma_create", "gpma_create_raw", "gpma_destro
            "gpma_cc_round", "gpma_pr_push", "gpma_pr_update", "gpma_pr_update_rows", "gpma_bfs_bits",
            "gpma_bfs_merge", "gpma_query_edges", "gpma_query_neighbors",
            "gpma_query_reachable", "gpma_debug_dump_aux", "gpma_dist_unique_id", "gpma_dist_create",
-           "gpma_dist_info", "gpma_pr_update_rows_dev", "gpma_validate_batch",
+           "gpma_dist_info", "gpma_pr_update_rows_dev", "gpma_validate_batch", "gpma_stats_host",
            "gpma_status_string", "gpma_last_error"]
 
 
@@ -312,6 +313,12 @@ class Gpma:
     def gpma_stats(self) -> dict:
         s = gpma_stats_t()
         self._check(lib().gpma_stats(self._h, C.byref(s)), "gpma_stats")
+        return {f: getattr(s, f) for f, _ in s._fields_}
+
+    def gpma_stats_host(self) -> dict:
+        """gpma_stats without device work (live_edges / tombstones not counted)."""
+        s = gpma_stats_t()
+        self._check(lib().gpma_stats_host(self._h, C.byref(s)), "gpma_stats_host")
         return {f: getattr(s, f) for f, _ in s._fields_}
 
     def gpma_debug_dump(self, keys=None, vals=None, row_offset=None, leaf_live=None, heads=None, stream=None):
