@@ -16,6 +16,7 @@ from paper_journals_pvldb_shalht17_b200 import Gpma  # noqa: E402
 
 ap = argparse.ArgumentParser()
 ap.add_argument("--grow", type=int, default=40)
+ap.add_argument("--shrink", type=int, default=30)
 a = ap.parse_args()
 dev = torch.device("cuda:0")
 cfg = CONFIGS[3]
@@ -46,7 +47,29 @@ with torch.cuda.stream(s):
             continue
         ins.append(e[0].elapsed_time(e[1]))
         dels.append(e[1].elapsed_time(e[2]))
+    sins, sdel = [], []
+    for step in range(a.shrink):
+        ik, iv = pool[b:b + (1 << 18)].contiguous(), vals[b:b + (1 << 18)].contiguous()
+        dk = pool[f:f + (1 << 20)].contiguous()
+        e = [torch.cuda.Event(enable_timing=True) for _ in range(3)]
+        e[0].record(s)
+        g.gpma_update_batch(ik, iv, 0, stream=s)
+        e[1].record(s)
+        g.gpma_update_batch(dk, None, 1, stream=s)
+        e[2].record(s)
+        e[2].synchronize()
+        b += 1 << 18
+        f += 1 << 20
+        r = g.gpma_stats()["resizes"]
+        if r != r0:
+            r0 = r
+            resz += 1
+            continue
+        sins.append(e[0].elapsed_time(e[1]))
+        sdel.append(e[1].elapsed_time(e[2]))
 h = len(ins) // 4
 print(json.dumps({"knobs": {k: v for k, v in os.environ.items() if k.startswith("GPMA_")},
-                  "insert_ms": float(np.mean(ins[h:])), "delete_ms": float(np.mean(dels[h:])),
-                  "steps": len(ins), "resizing_steps": resz}))
+                  "grow_insert_ms": float(np.mean(ins[h:])), "grow_delete_ms": float(np.mean(dels[h:])),
+                  "shrink_insert_ms": float(np.mean(sins)) if sins else None,
+                  "shrink_delete_ms": float(np.mean(sdel)) if sdel else None,
+                  "steps": len(ins) + len(sins), "resizing_steps": resz}))
