@@ -61,6 +61,7 @@ struct Ctrl {
   uint64_t ndirty;         // dirty windows recorded for the head fix-up
   uint64_t sum;            // scratch reductions
   uint64_t sum2;
+  uint64_t big;            // updates in leaf groups too large for the thread-per-group merge
 };
 
 // Per-level descriptors of one GPMA+ round (Alg. 4 l.7-15).

@@ -718,7 +718,7 @@ struct UpdDirect {              // a key-sorted batch (shared or global memory)
   __device__ uint32_t val(uint32_t j) const { return v[j]; }
 };
 
-template <class Upd>
+template <bool SORTED, class Upd>
 __device__ __forceinline__ LeafOut leaf_group_merge(uint64_t *rk, uint32_t *rv, uint32_t L, uint32_t t, uint32_t j0,
                                                     uint32_t j1, const Upd &U, uint32_t bound, uint32_t *keep,
                                                     const uint64_t *key, uint32_t *cnt, uint32_t *tmask,
@@ -733,7 +733,9 @@ __device__ __forceinline__ LeafOut leaf_group_merge(uint64_t *rk, uint32_t *rv, 
   for (uint32_t j = j0; j < j1; ++j) {
     const uint64_t uk = U.key(j);
     bool last = true;                                    // R10: a later copy in the group wins
-    for (uint32_t j2 = j + 1; j2 < j1 && last; ++j2) last = U.key(j2) != uk;
+    if (SORTED) last = j + 1 == j1 || U.key(j + 1) != uk;   // (key-sorted: copies are adjacent)
+    else
+      for (uint32_t j2 = j + 1; j2 < j1 && last; ++j2) last = U.key(j2) != uk;   // (groups <= IL_BIG)
     uint32_t h = 0;
     if (last) {
       ++o.effs;
@@ -805,6 +807,7 @@ __device__ __forceinline__ LeafOut leaf_group_merge(uint64_t *rk, uint32_t *rv, 
 }
 
 constexpr int ILU_T = 128;      // 4 warps: 4 x 32 leaves staged in shared memory
+constexpr uint32_t IL_BIG = 64;  // larger leaf groups take the key-sorted fallback (no O(u^2) dedupe)
 template <int L>
 __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
                                                     const uint64_t *__restrict__ tk, const uint32_t *__restrict__ tix,
@@ -813,7 +816,8 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
                                                     uint32_t *__restrict__ cnt, uint32_t *__restrict__ tmask,
                                                     uint64_t *__restrict__ head, uint64_t *__restrict__ row_offset,
                                                     uint32_t *__restrict__ deg, uint32_t rb, uint32_t bound,
-                                                    uint32_t *__restrict__ keep, uint2 *__restrict__ dirty, Ctrl *c) {
+                                                    uint32_t *__restrict__ keep, uint32_t *__restrict__ bigf,
+                                                    uint2 *__restrict__ dirty, Ctrl *c) {
   // Leaf I/O is warp-cooperative: the 32 leaves of a warp's 32 groups move through shared memory
   // in coalesced 16-B chunks (L/2 lanes per leaf for the keys, L/4 for the values), so a leaf is
   // whole 128-B lines instead of 32 single-sector requests per load instruction.
@@ -870,9 +874,19 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
     // the thread's leaf is its row of shared memory: dynamic indexing is free there, so the
     // merge is a few moves per update instead of static select networks over registers
     const UpdIdx U{ik, iv, tix};
-    const LeafOut lo_ = have ? leaf_group_merge(mk + lane * KS, mv + lane * KS, (uint32_t)L, t, j0, j1, U, bound, keep,
-                                                key, cnt, tmask, head, row_offset, deg, rb, dirty, c)
-                             : LeafOut{};
+    // an oversized group (> IL_BIG updates: an adversarial batch piling into one leaf) is left to
+    // the key-sorted fallback after the kernel; its updates are flagged in bigf
+    const bool big = have && j1 - j0 > IL_BIG;
+    if (have)
+      for (uint32_t j = j0; j < j1; ++j) {
+        bigf[j] = big ? 1u : 0u;
+        if (big) keep[j] = 0u;
+      }
+    if (big) atomicAdd((unsigned long long *)&c->big, (unsigned long long)(j1 - j0));
+    const LeafOut lo_ = have && !big ? leaf_group_merge<false>(mk + lane * KS, mv + lane * KS, (uint32_t)L, t, j0, j1, U,
+                                                               bound, keep, key, cnt, tmask, head, row_offset, deg,
+                                                               rb, dirty, c)
+                                     : LeafOut{};
     const bool ok = lo_.ok;
     const uint32_t hitm = lo_.hitm;
     news += lo_.nnew;
@@ -975,6 +989,7 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
     c->ndirty = 0;
     c->sum = 0;
     c->sum2 = 0;
+    c->big = 0;
     s_stats[0] = s_stats[1] = s_stats[2] = 0;
   }
   // validate (RESERVED beats RANGE; nothing is mutated on either)
@@ -1053,8 +1068,8 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
         rk[p] = key[lb + p];
         rv[p] = val[lb + p];
       }
-      const LeafOut o = leaf_group_merge(rk, rv, (uint32_t)L, t, j0, j1, U, bound, kp, key, cnt, tmask, head,
-                                         row_offset, deg, rb, dirty, c);
+      const LeafOut o = leaf_group_merge<true>(rk, rv, (uint32_t)L, t, j0, j1, U, bound, kp, key, cnt, tmask, head,
+                                               row_offset, deg, rb, dirty, c);
       if (o.ok)
         for (int p = 0; p < L; ++p) key[lb + p] = rk[p];
       if (o.ok || o.hitm)
@@ -3515,15 +3530,17 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
     GP_LAUNCH(g, k_gstart, grid_for(n), TB, 0, s, hf, gid, n, gstart, g->ctrl_d);
     const uint32_t bound = (uint32_t)g->tmax[0];
     uint2 *dirty = (uint2 *)g->b_dirty.p;
+    GP_CHECK(g, ensure(g, g->b_tgt, (n + 1) * 4, s));
+    uint32_t *bigf = (uint32_t *)g->b_tgt.p;
     if (g->L == 16)
       GP_LAUNCH(g, k_ins_leaf_u<16>, grid_for(n, ILU_T), ILU_T, 0, s, ik, iv, tk, tix, gstart, gid + n, g->key, g->val, g->cnt,
-                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, bigf, dirty, g->ctrl_d);
     else if (g->L == 8)
       GP_LAUNCH(g, k_ins_leaf_u<8>, grid_for(n, ILU_T), ILU_T, 0, s, ik, iv, tk, tix, gstart, gid + n, g->key, g->val, g->cnt,
-                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, bigf, dirty, g->ctrl_d);
     else
       GP_LAUNCH(g, k_ins_leaf_u<4>, grid_for(n, ILU_T), ILU_T, 0, s, ik, iv, tk, tix, gstart, gid + n, g->key, g->val, g->cnt,
-                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, dirty, g->ctrl_d);
+                tmask_of(g), g->head, g->row_offset, g->deg, g->rb, bound, keep, bigf, dirty, g->ctrl_d);
     GP_CHECK(g, scan_u32(g, keep, pos, n, s));
     GP_LAUNCH(g, k_upd_summary, 1, 1, 0, s, (const uint32_t *)nullptr, pos, n, g->ctrl_d);
     GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
@@ -3792,6 +3809,65 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   return update_after_prefix(g, ik, iv, n, op, path, srt, s);
 }
 
+__global__ void k_big_gather(const uint32_t *__restrict__ bigf, const uint32_t *__restrict__ bpos, uint64_t n,
+                             const uint32_t *__restrict__ tix, const uint64_t *__restrict__ ik,
+                             const uint32_t *__restrict__ iv, uint64_t *__restrict__ bk, uint32_t *__restrict__ bv) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < n; j += (uint64_t)gridDim.x * blockDim.x)
+    if (bigf[j]) {
+      const uint32_t i = tix[j];
+      bk[bpos[j]] = ik[i];
+      bv[bpos[j]] = iv[i];
+    }
+}
+
+__global__ void k_iota(uint32_t *__restrict__ out, uint64_t n, uint32_t base) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < n; j += (uint64_t)gridDim.x * blockDim.x)
+    out[j] = base + (uint32_t)j;
+}
+
+// Level 0 for the updates of oversized leaf groups (flagged by k_ins_leaf_u in b_tgt): compact,
+// sort by key (stable: copies adjacent, the last wins, R10), locate, group, merge with the
+// sub-warp leaf kernel (any group size); the rejected keys are appended to the pending list at
+// (pk, pv, pt, seq) with sequence numbers from seq0.  The control block keeps accumulating.
+static gpma_status big_groups(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, const Sorted &srt,
+                              uint64_t nbig, uint64_t *pk, uint32_t *pv, uint32_t *pt, uint32_t *seq, uint64_t seq0,
+                              uint64_t *p2, cudaStream_t s) {
+  const uint64_t nl = g->cap / g->L;
+  const uint64_t *ro = g->rows_indexed ? g->row_offset : nullptr;
+  uint32_t *bigf = (uint32_t *)g->b_tgt.p, *bpos = (uint32_t *)g->b_kpos.p;
+  GP_CHECK(g, scan_u32(g, bigf, bpos, n, s));
+  GP_CHECK(g, ensure(g, g->b_stage[2], nbig * 8 + 16, s));
+  GP_CHECK(g, ensure(g, g->b_stage[3], nbig * 4 + 16, s));
+  uint64_t *bk = (uint64_t *)g->b_stage[2].p;
+  uint32_t *bv = (uint32_t *)g->b_stage[3].p;
+  GP_LAUNCH(g, k_big_gather, grid_for(n), TB, 0, s, bigf, bpos, n, (const uint32_t *)srt.v, ik, iv, bk, bv);
+  Sorted s2;
+  gpma_status st = sort_batch(g, bk, bv, nbig, &s2, s);
+  if (st) return st;
+  uint32_t *tgt = bigf, *hf = (uint32_t *)g->b_acc.p, *gid = bpos, *gstart = (uint32_t *)g->b_wfirst.p;
+  uint32_t *keep = (uint32_t *)g->b_keep.p, *pos = (uint32_t *)g->b_pos.p;
+  GP_LAUNCH(g, k_locate, grid_for(nbig, LOC_T), LOC_T, 0, s, s2.k, nbig, g->head, (uint32_t)nl, g->L, g->rb, ro, tgt, hf,
+            g->ctrl_d);
+  GP_CHECK(g, scan_u32(g, hf, gid, nbig, s));
+  GP_LAUNCH(g, k_gstart, grid_for(nbig), TB, 0, s, hf, gid, nbig, gstart, g->ctrl_d);
+  GP_LAUNCH(g, k_ins_leaf, grid_for((nbig + 31) / 32 * 32, IL_T), IL_T, 0, s, s2.k, s2.v, tgt, gstart, gid + nbig,
+            g->key, g->val, g->cnt, tmask_of(g), g->head, g->row_offset, g->deg, g->rb, g->L, (uint32_t)g->tmax[0], keep,
+            (uint2 *)g->b_dirty.p, g->ctrl_d);
+  GP_CHECK(g, scan_u32(g, keep, pos, nbig, s));
+  GP_CHECK(g, readback(g, g->pin, pos + nbig, 4, s));
+  GP_CHECK(g, readback(g, g->ctrl_h, g->ctrl_d, sizeof(Ctrl), s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  uint32_t m;
+  memcpy(&m, g->pin, 4);
+  *p2 = m;
+  if (m) {
+    GP_LAUNCH(g, k_compact_pending, grid_for(nbig), TB, 0, s, keep, pos, nbig, s2.k, s2.v, tgt, pk, pv, pt, g->ctrl_d);
+    GP_LAUNCH(g, k_iota, grid_for(m), TB, 0, s, seq, (uint64_t)m, (uint32_t)seq0);
+  }
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 // After the prefix's host round trip: the pending list of level 1 (if any), the level loop, the
 // root resize, the head fix-up.  ik / iv: the batch the prefix read (staged or the caller's).
 static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int path,
@@ -3823,16 +3899,28 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
   } else if (path == PATH_INS_LEAF) {
     // pending after level 0: the new keys the leaves rejected, gathered in leaf order, then put
     // in key order (the level loop's pending lists are key-sorted, Alg. 4 l.12-15)
-    const uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
+    uint64_t p_new = (uint32_t)g->ctrl_h->sum2;
+    uint64_t *pk1 = (uint64_t *)g->b_pk[1].p;
+    uint32_t *pv1 = (uint32_t *)g->b_pv[1].p, *pt1 = (uint32_t *)g->b_pt[1].p, *seq = (uint32_t *)g->b_keep2.p;
+    if (p_new)
+      GP_LAUNCH(g, k_pend_gather, grid_for(n), TB, 0, s, (const uint32_t *)g->b_keep.p, (const uint32_t *)g->b_pos.p,
+                n, (const uint32_t *)srt.v, (const uint64_t *)srt.k, ik, iv, pk1, pv1, pt1, seq);
+    if (g->ctrl_h->big) {
+      // oversized leaf groups (an adversarial batch piling into one leaf): the key-sorted fused
+      // path on their updates -- compacted in leaf order, which is arrival order inside a group
+      uint64_t p2 = 0;
+      if ((st = big_groups(g, ik, iv, n, srt, g->ctrl_h->big, pk1 + p_new, pv1 + p_new, pt1 + p_new, seq + p_new,
+                           p_new, &p2, s)))
+        return st;
+      p_new += p2;
+      g->last.last_unique = g->ctrl_h->nunique;
+      g->last.last_pending = (uint32_t)g->ctrl_h->sum;
+    }
     dirty_base = g->ctrl_h->ndirty;
     g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;
     g->last.last_windows_rewritten += g->ctrl_h->windows_rewritten;
     g->last.last_level0_windows = g->ctrl_h->windows_rewritten;
     if (p_new) {
-      uint64_t *pk1 = (uint64_t *)g->b_pk[1].p;
-      uint32_t *pv1 = (uint32_t *)g->b_pv[1].p, *pt1 = (uint32_t *)g->b_pt[1].p, *seq = (uint32_t *)g->b_keep2.p;
-      GP_LAUNCH(g, k_pend_gather, grid_for(n), TB, 0, s, (const uint32_t *)g->b_keep.p, (const uint32_t *)g->b_pos.p,
-                n, (const uint32_t *)srt.v, (const uint64_t *)srt.k, ik, iv, pk1, pv1, pt1, seq);
       int sh[8], which = 0;
       const int ns = key_shifts(g->V, sh);
       GP_CHECK(g, radix_sort_pairs(g, pk1, seq, (uint64_t *)g->b_sk[1].p, (uint32_t *)g->b_sv[1].p, p_new, sh, ns, s,

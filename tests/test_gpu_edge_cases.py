@@ -157,3 +157,26 @@ def test_torch_allocator_hooks():
     end = torch.cuda.memory_allocated()
     assert mid - end >= cap * 12                                     # the store went back to torch
     assert end <= before + (2 << 20)                                 # (torch's own lazy state aside)
+
+
+@pytest.mark.parametrize("mode", [0, 1])
+def test_oversized_leaf_groups(mode):
+    """NEXT-4 adversarial batch: 30000 updates piling into two source rows (the leaf groups hold
+    thousands of updates, heavy duplication with distinct values, so the last copy must win), mixed
+    with ordinary random updates: the oversized groups take the key-sorted fallback, the rest the
+    thread-per-group merge -- one layout, equal to the oracle's."""
+    rng = np.random.default_rng(77)
+    V = 4096
+    k0 = ((rng.integers(0, V, 20000) << 32) | rng.integers(0, V, 20000)).astype(np.uint64).tolist()
+    g, o = _pair(V, k0, [1] * len(k0), delete_mode=mode)
+    hot = (np.repeat([7, 3001], 15000) << 32) | rng.integers(0, 6000, 30000) % V
+    rnd = (rng.integers(0, V, 5000) << 32) | rng.integers(0, V, 5000)
+    ks = np.concatenate([hot, rnd]).astype(np.uint64)
+    perm = rng.permutation(ks.size)
+    ks = ks[perm].tolist()
+    vs = rng.integers(0, 1 << 31, len(ks)).tolist()
+    _apply(g, o, ks, vs)
+    assert_same_csr(g, o)
+    _apply(g, o, ks[:8000], op=1)
+    _apply(g, o, ks[4000:12000], vs[4000:12000])
+    assert_same_csr(g, o)
