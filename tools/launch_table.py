@@ -12,7 +12,7 @@ ki, mi, vi, ii = h.index("Kernel Name"), h.index("Metric Name"), h.index("Metric
 per = collections.defaultdict(dict)
 for r in rows[hi + 1:]:
     per[int(r[ii])][r[mi]] = r[vi]
-    per[int(r[ii])]["name"] = r[ki]
+    per[int(r[ii])]["name"] = r[ki][5:] if r[ki].startswith("void ") else r[ki]
 ids = sorted(per)
 names = [per[i]["name"] for i in ids]
 starts = [i for i, n in enumerate(names) if n.startswith(first)]
