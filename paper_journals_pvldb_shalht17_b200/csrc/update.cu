@@ -3881,7 +3881,7 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
   uint64_t p = (uint32_t)g->ctrl_h->sum;
   g->last.last_unique = g->ctrl_h->nunique;
   g->last.last_pending = p;
-  if (p == 0) return GPMA_OK;
+  if (p == 0 && !g->ctrl_h->big) return GPMA_OK;       // (oversized leaf groups still to do)
   if (lock) return gpma_lock_insert(g, p, s);
   int cur = 0;
   uint64_t dirty_base = 0;
