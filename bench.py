@@ -238,7 +238,8 @@ def run_gpma(args, rank, world, lrank):
                 slide_log.append({"slide": i, "top_level": st_h["last_top_level"],
                                   "slots_rewritten": st_h["last_slots_rewritten"],
                                   "windows_rewritten": st_h["last_windows_rewritten"],
-                                  "pending_after_prepass": st_h["last_pending"], "resized": st_h["last_resized"],
+                                  "pending_after_prepass": st_h["last_pending"],
+                                  "pending_level1": st_h["last_pending_level1"], "resized": st_h["last_resized"],
                                   "capacity": st_h["capacity"]})
             if fan is None:                    # serial: one stream, phase by phase
                 g.gpma_bfs(root, lv, stream=s)

@@ -118,6 +118,7 @@ typedef struct {
   uint64_t total_delete_keys; /* keys of delete batches                                */
   uint64_t total_slots_rewritten;   /* sum of last_slots_rewritten                       */
   uint64_t total_windows_rewritten;
+  uint64_t last_pending_level1;    /* updates the leaves rejected (climbing to level 1)   */
 } gpma_stats_t;
 
 /* Fill *cfg with the defaults above. */

@@ -2159,16 +2159,14 @@ __global__ void k_lvl_summary(Lvl a, Ctrl *c) {
 }
 
 // ---- device-resident level loop (Alg. 4 l.4-15 above the leaves) ----------------------------
-// One cooperative kernel runs levels 1, 2, ... on the device while the pending list is small
-// (<= CL_MAXP) and the windows fit a CTA's shared memory (<= CL_MAXS slots, TryInsert+ at
-// block scale): per level, CTA 0 forms the segments (UniqueSegments = RLE + scan,
-// l.18-21), every warp counts a window and tests it (CountSegment + density, l.23-25), every
-// CTA merges and re-dispatches accepted windows in shared memory (l.26-27, R7), CTA 0 promotes
-// the rest (l.12-15) -- grid-wide barriers between the phases instead of a host round trip per
-// level.  It stops at the first level it cannot take; the host continues from there (larger
-// windows, the root resize).
+// One cooperative kernel runs levels 1, 2, ... on the device while the windows fit a CTA's
+// shared memory (<= CL_MAXS slots, TryInsert+ at block scale): per level, the
+// segments (UniqueSegments = RLE + a grid-wide scan, l.18-21), a warp per window counts and
+// tests it (CountSegment + density, l.23-25), a CTA per accepted window merges and re-dispatches
+// it in shared memory (l.26-27, R7), the rest is promoted by a second grid-wide scan (l.12-15) --
+// grid-wide barriers between the phases instead of a host round trip per level.  It stops at the
+// first level whose windows are larger; the host continues from there (the root resize).
 constexpr int CL_T = 512, CL_I = 16;
-constexpr uint32_t CL_MAXP = CL_T * CL_I;            // 8192 pending updates
 constexpr uint32_t CL_MAXS = 4096;                   // slots of the largest window (48 KiB of keys + values)
 
 struct CoopState {
@@ -2183,6 +2181,7 @@ struct CoopArgs {
   uint32_t *pv[2], *pt[2];
   uint32_t *hf, *widx, *wfirst, *acc, *keep, *kpos;
   uint64_t *nw;
+  uint64_t *ctot;              // [gridDim] chunk totals of the grid-wide scans
   uint64_t *key;
   uint32_t *val, *cnt, *tmask;
   uint64_t *row_offset;
@@ -2231,80 +2230,104 @@ __device__ __forceinline__ uint64_t cl_scan(uint64_t (&v)[CL_I], uint64_t *wsum)
   return total;
 }
 
-// CTA 0: the segments of level S.lvl over the pending list S.cur (hf, widx, wfirst, q)
-__device__ void cl_segments(const CoopArgs &a, CoopState &S, uint64_t *wsum) {
-  const uint64_t p = S.p;
-  const uint32_t lvl = S.lvl;
-  const uint32_t *pt = a.pt[S.cur];
-  const uint64_t j0 = (uint64_t)threadIdx.x * CL_I;
-  uint64_t f[CL_I], e[CL_I];
+// Grid-wide exclusive scan of the 0/1 flags f(j), j < p (every CTA takes a contiguous chunk;
+// chunk scans, one barrier, the CTA totals' prefix, one barrier): out[j] = the prefix, returns the
+// total on every CTA.  flag_out (optional) receives the flags.
+template <class F>
+__device__ uint64_t cl_grid_scan(cooperative_groups::grid_group &grid, uint64_t p, const F &f, uint32_t *out,
+                                 uint32_t *flag_out, uint64_t *ctot, uint64_t *wsum) {
+  const uint64_t per = (p + gridDim.x - 1) / gridDim.x;
+  const uint64_t b0 = min(p, (uint64_t)blockIdx.x * per), b1 = min(p, b0 + per);
+  uint64_t carry = 0;
+  for (uint64_t t0 = b0; t0 < b1; t0 += (uint64_t)CL_T * CL_I) {       // block-uniform
+    uint64_t v[CL_I], fl[CL_I];
 #pragma unroll
-  for (int i = 0; i < CL_I; ++i) {
-    const uint64_t j = j0 + i;
-    f[i] = (j < p && (j == 0 || (pt[j] >> lvl) != (pt[j - 1] >> lvl))) ? 1u : 0u;
-    if (j < p) a.hf[j] = (uint32_t)f[i];
-    e[i] = f[i];
-  }
-  const uint64_t q = cl_scan(e, wsum);
-#pragma unroll
-  for (int i = 0; i < CL_I; ++i) {
-    const uint64_t j = j0 + i;
-    if (j < p) {
-      a.widx[j] = (uint32_t)e[i];
-      if (f[i]) a.wfirst[e[i]] = (uint32_t)j;
+    for (int i = 0; i < CL_I; ++i) {
+      const uint64_t j = t0 + (uint64_t)threadIdx.x * CL_I + i;
+      fl[i] = j < b1 ? f(j) : 0u;
+      v[i] = fl[i];
     }
+    const uint64_t tot = cl_scan(v, wsum);
+#pragma unroll
+    for (int i = 0; i < CL_I; ++i) {
+      const uint64_t j = t0 + (uint64_t)threadIdx.x * CL_I + i;
+      if (j < b1) {
+        out[j] = (uint32_t)(carry + v[i]);
+        if (flag_out) flag_out[j] = (uint32_t)fl[i];
+      }
+    }
+    carry += tot;
   }
-  if (threadIdx.x == 0) {
-    a.widx[p] = (uint32_t)q;
-    a.wfirst[q] = (uint32_t)p;
-    S.q = (uint32_t)q;
+  if (threadIdx.x == 0) ctot[blockIdx.x] = carry;
+  grid.sync();
+  uint64_t pre = 0, all = 0;
+  for (uint32_t k = threadIdx.x; k < gridDim.x; k += CL_T) {
+    const uint64_t x = ctot[k];
+    all += x;
+    if (k < blockIdx.x) pre += x;
   }
+  for (int o = 16; o; o >>= 1) {
+    pre += __shfl_xor_sync(0xffffffffu, pre, o);
+    all += __shfl_xor_sync(0xffffffffu, all, o);
+  }
+  __shared__ uint64_t s_pre[CL_T / 32], s_all[CL_T / 32];
+  if ((threadIdx.x & 31) == 0) {
+    s_pre[threadIdx.x >> 5] = pre;
+    s_all[threadIdx.x >> 5] = all;
+  }
+  __syncthreads();
+  pre = 0;
+  all = 0;
+  for (int k = 0; k < CL_T / 32; ++k) {
+    pre += s_pre[k];
+    all += s_all[k];
+  }
+  __syncthreads();
+  if (pre)
+    for (uint64_t j = b0 + threadIdx.x; j < b1; j += CL_T) out[j] += (uint32_t)pre;
+  return all;
 }
 
-// CTA 0: promote the rejected updates of the level to the next buffer (l.12-15), next level
-__device__ void cl_promote(const CoopArgs &a, CoopState &S, uint64_t *wsum) {
-  const uint64_t p = S.p;
-  const uint32_t cur = S.cur;
-  const uint64_t j0 = (uint64_t)threadIdx.x * CL_I;
-  uint64_t k[CL_I], kk[CL_I];
-#pragma unroll
-  for (int i = 0; i < CL_I; ++i) {
-    const uint64_t j = j0 + i;
-    k[i] = 0;
-    if (j < p) {
-      const uint32_t w = a.widx[j] + a.hf[j] - 1;
-      k[i] = a.acc[w] ? 0u : 1u;
+// the segments of level lvl over the pending list of buffer cur: hf, widx, wfirst; returns q
+__device__ uint64_t cl_segments(cooperative_groups::grid_group &grid, const CoopArgs &a, uint64_t p, uint32_t cur,
+                                uint32_t lvl, uint64_t *wsum) {
+  const uint32_t *pt = a.pt[cur];
+  const auto f = [&](uint64_t j) -> uint64_t {
+    return (j == 0 || (pt[j] >> lvl) != (pt[j - 1] >> lvl)) ? 1u : 0u;
+  };
+  const uint64_t q = cl_grid_scan(grid, p, f, a.widx, a.hf, a.ctot, wsum);
+  grid.sync();                                           // widx / hf complete
+  for (uint64_t j = blockIdx.x * (uint64_t)CL_T + threadIdx.x; j < p; j += (uint64_t)gridDim.x * CL_T)
+    if (a.hf[j]) a.wfirst[a.widx[j]] = (uint32_t)j;
+  if (blockIdx.x == 0 && threadIdx.x == 0) {
+    a.widx[p] = (uint32_t)q;
+    a.wfirst[q] = (uint32_t)p;
+  }
+  return q;
+}
+
+// promote the rejected updates of the level to the other buffer (l.12-15); returns the count
+__device__ uint64_t cl_promote(cooperative_groups::grid_group &grid, const CoopArgs &a, uint64_t p, uint32_t cur,
+                               uint64_t *wsum) {
+  const auto f = [&](uint64_t j) -> uint64_t { return a.acc[a.widx[j] + a.hf[j] - 1] ? 0u : 1u; };
+  const uint64_t pn = cl_grid_scan(grid, p, f, a.kpos, nullptr, a.ctot, wsum);
+  grid.sync();                                           // kpos complete
+  for (uint64_t j = blockIdx.x * (uint64_t)CL_T + threadIdx.x; j < p; j += (uint64_t)gridDim.x * CL_T)
+    if (!a.acc[a.widx[j] + a.hf[j] - 1]) {
+      const uint32_t d = a.kpos[j];
+      a.pk[cur ^ 1][d] = a.pk[cur][j];
+      a.pv[cur ^ 1][d] = a.pv[cur][j];
+      a.pt[cur ^ 1][d] = a.pt[cur][j];
     }
-    kk[i] = k[i];
-  }
-  const uint64_t pn = cl_scan(kk, wsum);
-#pragma unroll
-  for (int i = 0; i < CL_I; ++i) {
-    const uint64_t j = j0 + i;
-    if (j < p && k[i]) {
-      a.pk[cur ^ 1][kk[i]] = a.pk[cur][j];
-      a.pv[cur ^ 1][kk[i]] = a.pv[cur][j];
-      a.pt[cur ^ 1][kk[i]] = a.pt[cur][j];
-    }
-  }
-  __syncthreads();
-  if (threadIdx.x == 0) {
-    S.top = S.lvl;
-    S.p = pn;
-    if (pn) S.cur = cur ^ 1;
-    S.lvl += 1;
-    S.done = (pn == 0 || S.lvl > a.h || ((uint64_t)a.L << S.lvl) > CL_MAXS) ? 1u : 0u;
-  }
-  __syncthreads();
-  __threadfence_block();
+  return pn;
 }
 
 // one accepted window merged and re-dispatched in shared memory (CTA-wide, Alg. 4 l.26-27)
-__device__ void cl_merge_window(const CoopArgs &a, const CoopState &S, uint32_t w, uint64_t *mk, uint32_t *mv,
+__device__ void cl_merge_window(const CoopArgs &a, uint32_t cur, uint32_t lvl, uint32_t w, uint64_t *mk, uint32_t *mv,
                                 uint32_t *lpre) {
-  const uint32_t lvl = S.lvl, L = a.L;
-  const uint64_t *pk = a.pk[S.cur];
-  const uint32_t *pv = a.pv[S.cur], *pt = a.pt[S.cur];
+  const uint32_t L = a.L;
+  const uint64_t *pk = a.pk[cur];
+  const uint32_t *pv = a.pv[cur], *pt = a.pt[cur];
   const uint32_t Lc = 1u << lvl, ws = L << lvl;
   const uint64_t leaf0 = ((uint64_t)(pt[a.wfirst[w]] >> lvl)) << lvl;
   const uint64_t N = a.nw[w];
@@ -2411,14 +2434,14 @@ __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
   __shared__ uint64_t wsum[CL_T / 32];
   cooperative_groups::grid_group grid = cooperative_groups::this_grid();
   CoopState &S = *a.st;
-  if (blockIdx.x == 0) cl_segments(a, S, wsum);
-  grid.sync();
+  // every CTA follows the same state: (p, cur, lvl) are recomputed identically everywhere
+  uint64_t p = S.p;
+  uint32_t cur = S.cur, lvl = S.lvl;
   uint64_t wins = 0, slots = 0;
-  while (true) {
-    const uint32_t done = *(volatile uint32_t *)&S.done;
-    if (done) break;
-    const uint32_t lvl = *(volatile uint32_t *)&S.lvl, q = *(volatile uint32_t *)&S.q;
-    const uint32_t cur = *(volatile uint32_t *)&S.cur;
+  uint32_t top = lvl;
+  while (p > 0 && lvl <= a.h && ((uint64_t)a.L << lvl) <= CL_MAXS) {
+    const uint64_t q = cl_segments(grid, a, p, cur, lvl, wsum);
+    grid.sync();
     const uint32_t *pt = a.pt[cur];
     // CountSegment + CountUpdatesInSegment + density test: a warp per window
     {
@@ -2440,22 +2463,30 @@ __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
     }
     grid.sync();
     // Merge + re-dispatch evenly: a CTA per accepted window
-    for (uint32_t w = blockIdx.x; w < q; w += gridDim.x) {
+    for (uint64_t w = blockIdx.x; w < q; w += gridDim.x) {
       if (!a.acc[w]) continue;
-      cl_merge_window(a, S, w, mk, mv, lpre);
+      cl_merge_window(a, cur, lvl, (uint32_t)w, mk, mv, lpre);
       ++wins;
       slots += (uint64_t)a.L << lvl;
     }
     grid.sync();
-    if (blockIdx.x == 0) {
-      cl_promote(a, S, wsum);
-      if (!S.done) cl_segments(a, S, wsum);
-    }
-    grid.sync();
+    const uint64_t pn = cl_promote(grid, a, p, cur, wsum);
+    grid.sync();                                         // the next buffer is complete
+    top = lvl;
+    p = pn;
+    if (pn) cur ^= 1u;
+    ++lvl;
   }
   if (threadIdx.x == 0 && wins) {
     atomicAdd((unsigned long long *)&S.windows, (unsigned long long)wins);
     atomicAdd((unsigned long long *)&S.slots, (unsigned long long)slots);
+  }
+  if (blockIdx.x == 0 && threadIdx.x == 0) {
+    S.p = p;
+    S.cur = cur;
+    S.lvl = lvl;
+    S.top = top;
+    S.done = 1;
   }
 }
 
@@ -3142,7 +3173,8 @@ __global__ void k_coop_init(CoopState *st, uint64_t p, uint32_t cur, uint32_t lv
 static bool coop_eligible(gpma *g, uint64_t p, uint32_t lvl) {
   const char *e = getenv("GPMA_LVL_COOP");
   if (e && atoi(e) == 0) return false;
-  return p <= CL_MAXP && ((uint64_t)g->L << lvl) <= CL_MAXS && g->h < 48;
+  (void)p;
+  return ((uint64_t)g->L << lvl) <= CL_MAXS && g->h < 48;
 }
 
 static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, uint64_t *dirty_base, int op,
@@ -3154,7 +3186,7 @@ static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, ui
     cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_levels_coop, CL_T, smem);
     return b > 0 ? b : 1;
   }();
-  GP_CHECK(g, ensure(g, g->b_misc2, sizeof(CoopState) + 64, s));
+  GP_CHECK(g, ensure(g, g->b_misc2, sizeof(CoopState) + 64 + (size_t)8 * 64 * 1024, s));
   CoopArgs a{};
   for (int i = 0; i < 2; ++i) {
     a.pk[i] = (uint64_t *)g->b_pk[i].p;
@@ -3184,6 +3216,7 @@ static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, ui
     a.tmax[i] = g->tmax[i];
   }
   a.st = (CoopState *)g->b_misc2.p;
+  a.ctot = (uint64_t *)((char *)g->b_misc2.p + ((sizeof(CoopState) + 63) & ~(size_t)63));
   a.c = g->ctrl_d;
   GP_LAUNCH(g, k_coop_init, 1, 1, 0, s, a.st, p, (uint32_t)cur, lvl, g->ctrl_d, *dirty_base);
   const int grid = std::max(1, std::min(blocks_per_sm * num_sms(), 4 * num_sms()));
@@ -3965,6 +3998,7 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     p = p_new;
     lvl = 1;
   }
+  if (lvl == 1) g->last.last_pending_level1 = p;
   if (p > 0 && lvl >= 1 && lvl <= g->h && !g->trace_on && coop_eligible(g, p, lvl)) {
     Nvtx nv("update: device level loop");
     if ((st = coop_levels(g, cur, p, lvl, &dirty_base, op, s))) return st;
