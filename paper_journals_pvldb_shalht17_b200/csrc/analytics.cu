@@ -156,10 +156,12 @@ __global__ void k_bfs_frontier(const int32_t *__restrict__ levels, uint32_t V, i
 }
 
 // frontier list from the bitmap (sparse levels only: few set bits)
+// (zero != nullptr: also clears the next level's frontier bitmap, same word range -- one launch less)
 __global__ void k_bfs_list(const uint32_t *__restrict__ bm, uint32_t nwords, uint32_t *__restrict__ list,
-                           uint32_t *n) {
+                           uint32_t *n, uint32_t *__restrict__ zero) {
   for (uint64_t w = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; w < nwords;
        w += (uint64_t)gridDim.x * blockDim.x) {
+    if (zero) zero[w] = 0u;
     uint32_t b = bm[w];
     if (!b) continue;
     uint32_t base = atomicAdd(n, (uint32_t)__popc(b));
@@ -242,9 +244,14 @@ __global__ void __launch_bounds__(TA) k_bfs_expand(const uint32_t *__restrict__ 
 constexpr int BFS_LA_K = 4;
 __global__ void __launch_bounds__(TA) k_bfs_leaf_active(const uint64_t *__restrict__ head, uint64_t nleaves,
                                                         uint32_t V, const uint32_t *__restrict__ bm,
-                                                        uint32_t *__restrict__ alist, uint32_t *__restrict__ nact) {
+                                                        uint32_t *__restrict__ alist, uint32_t *__restrict__ nact,
+                                                        uint32_t *__restrict__ zero, uint32_t zwords) {
   static_assert(BFS_LA_K * (TA / 32) == 32, "one warp scans the per-warp counts");
   __shared__ uint32_t wofs[BFS_LA_K * (TA / 32)];
+  if (zero)                                              // the next level's frontier bitmap
+    for (uint64_t w = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; w < zwords;
+         w += (uint64_t)gridDim.x * blockDim.x)
+      zero[w] = 0u;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint64_t per = (uint64_t)TA * BFS_LA_K;
   for (uint64_t b0 = blockIdx.x * per; b0 < nleaves; b0 += (uint64_t)gridDim.x * per) {
@@ -331,6 +338,13 @@ static uint32_t bfs_sparse_f() {
   return e ? (uint32_t)atol(e) : 32768u;
 }
 
+// read back nwords words to pinned host memory, then clear zwords words at zero (one launch)
+__global__ void k_readback_zero(uint32_t *dst, const uint32_t *src, uint32_t nwords, uint32_t *zero, uint32_t zwords) {
+  for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) dst[i] = src[i];
+  __syncwarp();
+  for (uint32_t i = threadIdx.x; i < zwords; i += blockDim.x) zero[i] = 0u;
+}
+
 gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
   GP_LAUNCH(g, k_bfs_init, grid_for(g->V), TA, 0, s, levels, g->V, root);
   GP_CHECK(g, cudaGetLastError());
@@ -341,7 +355,8 @@ gpma_status bfs_init(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
 // frontier list; dense -- sweep of the active leaves.  Discoveries get `depth`; with bm_next
 // they are also marked there and counted into *fnext (device).
 static gpma_status bfs_expand_level(gpma *g, Scratch &X, int32_t *levels, int32_t depth, const uint32_t *bm,
-                                    uint32_t F, uint32_t *bm_next, uint32_t *fnext, cudaStream_t s) {
+                                    uint32_t F, uint32_t *bm_next, uint32_t *fnext, cudaStream_t s,
+                                    uint32_t *zero_next = nullptr, bool cnt_zeroed = false) {
   const uint64_t V = g->V, nl = g->cap / g->L;
   GP_CHECK(g, ensure(g, X.b[0], (V + 1) * 4, s));
   GP_CHECK(g, ensure(g, X.misc, (nl + 2) * 4, s));
@@ -349,17 +364,18 @@ static gpma_status bfs_expand_level(gpma *g, Scratch &X, int32_t *levels, int32_
   uint32_t *alist = (uint32_t *)X.misc.p;
   uint32_t *cnt_d = reinterpret_cast<uint32_t *>(&X.ctrl_d->sum2);   // list / active-leaf count
   const uint32_t *tmask = tmask_of(g);
-  GP_CHECK(g, fill_zero(g, cnt_d, 4, s));
+  if (!cnt_zeroed) GP_CHECK(g, fill_zero(g, cnt_d, 4, s));
   if (F <= bfs_sparse_f()) {
     GP_CHECK(g, ensure(g, X.b[2], ((uint64_t)bfs_sparse_f() + 2) * 8, s));   // fixed size: no regrowth per level
     uint64_t *off = (uint64_t *)X.b[2].p;
-    GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, cnt_d);
+    GP_LAUNCH(g, k_bfs_list, grid_for((V + 31) / 32), TA, 0, s, bm, (uint32_t)((V + 31) / 32), list, cnt_d, zero_next);
     GP_LAUNCH(g, k_bfs_rowlen, grid_for(F), TA, 0, s, list, F, g->row_offset, g->rb, g->nr, off);
     GP_CHECK(g, scan_u64(g, off, off, F, s));
     GP_LAUNCH(g, k_bfs_expand, grid_cap(), TA, 0, s, list, F, off, g->row_offset, g->key, tmask, g->L,
               levels, depth, g->rb, bm_next, fnext);
   } else {
-    GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, alist, cnt_d);
+    GP_LAUNCH(g, k_bfs_leaf_active, grid_for(nl), TA, 0, s, g->head, nl, (uint32_t)V, bm, alist, cnt_d, zero_next,
+              (uint32_t)((V + 31) / 32 + 1));
     GP_LAUNCH(g, k_bfs_sweep, grid_cap(), TA, 0, s, g->key, tmask, g->L, alist, cnt_d, bm, levels, depth,
               bm_next, fnext);
   }
@@ -434,12 +450,16 @@ gpma_status bfs(gpma *g, uint32_t root, int32_t *levels, cudaStream_t s) {
   GP_LAUNCH(g, k_bfs_set_bit, 1, 32, 0, s, bm[0], root);
   uint32_t F = 1;
   int cur = 0;
+  // per level: the expansion kernels clear the next frontier bitmap themselves and the read-back
+  // of the frontier size clears the level counters (k_readback_zero) -- no zero-fill launches
+  GP_CHECK(g, fill_zero(g, &X.ctrl_d->sum, 16, s));     // F_d and the list / active-leaf counter
   for (int32_t depth = 1; F; ++depth, cur ^= 1) {
-    GP_CHECK(g, fill_zero(g, bm[cur ^ 1], words * 4, s));
-    GP_CHECK(g, fill_zero(g, F_d, 4, s));
-    gpma_status st = bfs_expand_level(g, X, levels, depth, bm[cur], F, bm[cur ^ 1], F_d, s);
+    gpma_status st = bfs_expand_level(g, X, levels, depth, bm[cur], F, bm[cur ^ 1], F_d, s, bm[cur ^ 1], true);
     if (st) return st;
-    GP_CHECK(g, readback(g, &X.ctrl_h->sum, F_d, 4, s));
+    g->launches++;
+    k_readback_zero<<<1, 32, 0, s>>>((uint32_t *)&X.ctrl_h->sum, (const uint32_t *)F_d, 1u,
+                                     (uint32_t *)&X.ctrl_d->sum, 4u);
+    GP_CHECK(g, cudaGetLastError());
     GP_CHECK(g, cudaStreamSynchronize(s));
     F = (uint32_t)(X.ctrl_h->sum & 0xFFFFFFFFu);
   }
