@@ -2189,6 +2189,7 @@ struct CoopArgs {
   uint64_t nleaves;
   uint32_t L, h, rb;
   int op;
+  int warp_merge;              // small windows merged by a warp (GPMA_LVL_WARP, default on)
   uint64_t tmin[48], tmax[48];
   CoopState *st;
   Ctrl *c;
@@ -2426,6 +2427,111 @@ __device__ void cl_merge_window(const CoopArgs &a, uint32_t cur, uint32_t lvl, u
   __syncthreads();                                       // the smem list is reused by the next window
 }
 
+// One accepted SMALL window (<= CL_WMAX slots: levels 1-4 at L = 16) merged and re-dispatched
+// by ONE WARP in its private shared-memory list: a CTA per 32-slot window (the block path above)
+// left 15 of 16 warps idle and made the level-1 step of a 1M batch with 10^4 rejected keys the
+// longest part of the insert.
+constexpr uint32_t CL_WMAX = 256;
+__device__ void cl_merge_window_warp(const CoopArgs &a, uint32_t cur, uint32_t lvl, uint32_t w, uint64_t *mk,
+                                     uint32_t *mv) {
+  const uint32_t L = a.L;
+  const uint64_t *pk = a.pk[cur];
+  const uint32_t *pv = a.pv[cur], *pt = a.pt[cur];
+  const uint32_t Lc = 1u << lvl, ws = L << lvl;
+  const uint64_t leaf0 = ((uint64_t)(pt[a.wfirst[w]] >> lvl)) << lvl;
+  const uint64_t N = a.nw[w];
+  const uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = (1u << lane) - 1u;
+  const uint32_t leafmask = (L == 32 ? 0xffffffffu : ((1u << L) - 1u) << (lane & ~(L - 1)));
+  // live entries before each leaf (Lc <= 32 leaves: one lane each, a warp scan)
+  const uint32_t c0 = (uint32_t)lane < Lc ? a.cnt[leaf0 + lane] : 0u;
+  uint32_t x = c0;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if (lane >= o) x += y;
+  }
+  const uint32_t lpre_me = x - c0;                       // lane l: live entries before leaf l
+  for (uint32_t o0 = 0; o0 < ws; o0 += 32) {             // gather the live entries
+    const uint32_t off = o0 + lane;
+    uint64_t k = KEY_NONE;
+    uint32_t v = 0;
+    if (off < ws) {
+      k = a.key[leaf0 * L + off];
+      v = a.val[leaf0 * L + off];
+    }
+    const bool live = off < ws && k != KEY_NONE && v != VAL_TOMB;
+    const uint32_t bal = __ballot_sync(0xffffffffu, live);
+    const uint32_t lidx = off / L;
+    const uint32_t lp = __shfl_sync(0xffffffffu, lpre_me, (int)(lidx & 31));
+    if (live) {
+      const uint64_t rl = __popc(bal & leafmask & lt) + lp;
+      const uint64_t cc = lower_bound_u64(pk, ub, ue, k) - ub;
+      bool drop = false;
+      uint64_t r;
+      if (a.op == GPMA_INSERT) {
+        r = rl + cc;
+      } else {
+        drop = (ub + cc < ue) && pk[ub + cc] == k;
+        r = rl - cc;
+      }
+      if (!drop) {
+        mk[r] = k;
+        mv[r] = v;
+      }
+    }
+  }
+  if (a.op == GPMA_INSERT) {                             // place the window's insertions
+    for (uint64_t j = ub + lane; j < ue; j += 32) {
+      const uint64_t k = pk[j];
+      const uint32_t t = pt[j];
+      uint64_t rl = 0;
+      {
+        // live entries of the window's leaves before t: the prefix held by lane (t - leaf0)
+        const uint32_t li = (uint32_t)(t - leaf0);
+        for (uint32_t l = 0; l < li; ++l) rl += a.cnt[leaf0 + l];
+      }
+      const uint64_t base = (uint64_t)t * L;
+      for (uint32_t q = 0; q < L; ++q) {
+        const uint64_t xk = a.key[base + q];
+        if (xk == KEY_NONE || xk > k) break;
+        if (a.val[base + q] != VAL_TOMB) ++rl;
+      }
+      const uint64_t r = (j - ub) + rl;
+      mk[r] = k;
+      mv[r] = pv[j];
+    }
+  }
+  __syncwarp();                                          // every read of the window is done
+  for (uint32_t off = lane; off < ws; off += 32) {       // re-dispatch evenly (R7)
+    const uint64_t l = leaf_div(off, L), q = leaf_mod(off, L);
+    const uint64_t lo = l * N / Lc, hi = (l + 1) * N / Lc;
+    const uint64_t sl = leaf0 * L + off;
+    if (q < hi - lo) {
+      const uint64_t k = mk[lo + q];
+      a.key[sl] = k;
+      a.val[sl] = mv[lo + q];
+      if (is_guard_key(k)) a.row_offset[(k >> 32) - a.rb + 1] = sl;
+    } else {
+      a.key[sl] = KEY_NONE;
+      a.val[sl] = 0;
+    }
+    if (q == 0) {
+      a.cnt[leaf0 + l] = (uint32_t)(hi - lo);
+      a.tmask[leaf0 + l] = 0u;
+      uint32_t gc = 0;
+      for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(mk[e]);
+      a.tmask[a.nleaves + leaf0 + l] = gc;
+    }
+  }
+  if (lane == 0) {
+    const uint64_t d = atomicAdd((unsigned long long *)&a.c->ndirty, 1ull);
+    a.dirty[d] = make_uint2((uint32_t)leaf0, Lc);
+  }
+  __syncwarp();                                          // the warp's list is reused by its next window
+}
+
 __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
   extern __shared__ __align__(16) unsigned char cl_smem[];
   uint64_t *mk = reinterpret_cast<uint64_t *>(cl_smem);
@@ -2462,12 +2568,29 @@ __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
       }
     }
     grid.sync();
-    // Merge + re-dispatch evenly: a CTA per accepted window
-    for (uint64_t w = blockIdx.x; w < q; w += gridDim.x) {
-      if (!a.acc[w]) continue;
-      cl_merge_window(a, cur, lvl, (uint32_t)w, mk, mv, lpre);
-      ++wins;
-      slots += (uint64_t)a.L << lvl;
+    // Merge + re-dispatch evenly: a warp per accepted small window, a CTA per larger one
+    if (((uint64_t)a.L << lvl) <= CL_WMAX && a.L <= 32 && lvl <= 5 && a.warp_merge) {
+      const uint32_t wi = threadIdx.x >> 5;
+      uint64_t *wk_ = mk + (uint64_t)wi * CL_WMAX;
+      uint32_t *wv_ = reinterpret_cast<uint32_t *>(mk + (uint64_t)(CL_T / 32) * CL_WMAX) + (uint64_t)wi * CL_WMAX;
+      const uint64_t nwarps = (uint64_t)gridDim.x * (CL_T / 32);
+      for (uint64_t w = (blockIdx.x * (uint64_t)CL_T + threadIdx.x) / 32; w < q; w += nwarps) {
+        if (!a.acc[w]) continue;
+        cl_merge_window_warp(a, cur, lvl, (uint32_t)w, wk_, wv_);
+        if ((threadIdx.x & 31) == 0) {
+          ++wins;
+          slots += (uint64_t)a.L << lvl;
+        }
+      }
+    } else {
+      for (uint64_t w = blockIdx.x; w < q; w += gridDim.x) {
+        if (!a.acc[w]) continue;
+        cl_merge_window(a, cur, lvl, (uint32_t)w, mk, mv, lpre);
+        if (threadIdx.x == 0) {
+          ++wins;
+          slots += (uint64_t)a.L << lvl;
+        }
+      }
     }
     grid.sync();
     const uint64_t pn = cl_promote(grid, a, p, cur, wsum);
@@ -2477,7 +2600,7 @@ __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
     if (pn) cur ^= 1u;
     ++lvl;
   }
-  if (threadIdx.x == 0 && wins) {
+  if (wins) {
     atomicAdd((unsigned long long *)&S.windows, (unsigned long long)wins);
     atomicAdd((unsigned long long *)&S.slots, (unsigned long long)slots);
   }
@@ -3211,6 +3334,10 @@ static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, ui
   a.h = g->h;
   a.rb = g->rb;
   a.op = op;
+  {
+    const char *e = getenv("GPMA_LVL_WARP");          // read per call (tests flip it)
+    a.warp_merge = e ? atoi(e) : 1;
+  }
   for (uint32_t i = 0; i <= g->h; ++i) {
     a.tmin[i] = g->tmin[i];
     a.tmax[i] = g->tmax[i];

@@ -144,7 +144,7 @@ def test_config0_sliding_window_graph_replay(seed):
 
 
 @pytest.mark.parametrize("knob", ["GPMA_DEL_SORT=1", "GPMA_INS_FUSED=0", "GPMA_INS_LEAFSORT=0",
-                                  "GPMA_INS_LEAFSORT=0,GPMA_INS_THREAD=0", "GPMA_LVL_COOP=0", "GPMA_ILP=1",
+                                  "GPMA_INS_LEAFSORT=0,GPMA_INS_THREAD=0", "GPMA_LVL_COOP=0", "GPMA_LVL_WARP=0", "GPMA_ILP=1",
                                   "GPMA_ILP=4", "GPMA_SMALL=2048", "GPMA_SMALL=0,GPMA_DEL_SORT=1"])
 @pytest.mark.parametrize("seed", range(3))
 def test_config0_alternative_paths(seed, knob, monkeypatch):
@@ -298,13 +298,14 @@ def test_medium_rmat_multi_tile(mode):
     assert_pr_close(x32, xo, fp64=False, what="rmat-s16 fp32")
 
 
-@pytest.mark.parametrize("coop", ["1", "0"])
+@pytest.mark.parametrize("coop", ["1", "0", "1-blockmerge"])
 @pytest.mark.parametrize("mode", [0, 1])
 def test_sorted_stream_hot_window(coop, mode, monkeypatch):
     """Ascending-key batches concentrated in one region (NEXT-4 pattern): deep climbs through the
     device-resident level loop (coop=1: levels with windows <= 4096 slots in one cooperative
     kernel) or the host-driven one, then strict / lazy deletes of the hot keys."""
-    monkeypatch.setenv("GPMA_LVL_COOP", coop)
+    monkeypatch.setenv("GPMA_LVL_COOP", coop[0])
+    monkeypatch.setenv("GPMA_LVL_WARP", "0" if coop.endswith("blockmerge") else "1")
     V = 4096
     rng = np.random.default_rng(11)
     k0 = _keys(rng.integers(0, V, 20000), rng.integers(0, V, 20000))
