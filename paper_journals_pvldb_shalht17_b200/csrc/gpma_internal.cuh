@@ -54,7 +54,7 @@ struct DevBuf {
 // Device-side control block (counters written by kernels, read back in one copy).
 struct Ctrl {
   uint32_t err;            // validation bits: 1 = range, 2 = reserved
-  uint32_t pad0;
+  uint32_t seq;            // host mirror only: the call's sequence number, written last (wait_ctrl)
   uint64_t nunique;        // distinct keys in the batch
   uint64_t slots_rewritten;
   uint64_t windows_rewritten;
@@ -87,6 +87,85 @@ struct Scratch {
   Ctrl *ctrl_d = nullptr;
   Ctrl *ctrl_h = nullptr;         // pinned mirror
 };
+
+#ifdef __CUDACC__
+// Ascending sort of the (key, index) pairs sk/si[0, np2) in shared memory by one CTA (np2 a power
+// of two, 2 <= np2 <= 2 * blockDim.x; entries past the real ones hold padding keys): a bitonic
+// network with thread t holding elements 2t and 2t+1 in registers.  Strides 1..32 stay in
+// registers (in-thread, then warp shuffles -- no barrier), only strides >= 64 go through the
+// shared arrays (two barriers each): 15 of the 55 stages of a 1024-pair sort instead of all 55.
+// Ties on the key are broken by the index, so with distinct indices the order is total (stable
+// when the indices are the arrival positions).  Every thread of the CTA must call it.
+__device__ __forceinline__ bool cta_pair_less(uint64_t ka, uint32_t ia, uint64_t kb, uint32_t ib) {
+  return ka < kb || (ka == kb && ia < ib);
+}
+__device__ __forceinline__ void cta_pair_cas(uint64_t &k, uint32_t &x, uint64_t pk, uint32_t px, uint32_t i,
+                                             uint32_t j, uint32_t size) {
+  const bool up = (i & size) == 0;
+  const bool keep_min = (i < j) == up;
+  const bool own_less = cta_pair_less(k, x, pk, px);
+  if (keep_min != own_less) {
+    k = pk;
+    x = px;
+  }
+}
+__device__ inline void cta_bitonic_sort(uint64_t *sk, uint32_t *si, uint32_t np2) {
+  const uint32_t t = threadIdx.x;
+  const bool act = 2 * t < np2;
+  uint64_t k0 = ~0ull, k1 = ~0ull;
+  uint32_t x0 = ~0u, x1 = ~0u;
+  if (act) {
+    k0 = sk[2 * t];
+    x0 = si[2 * t];
+    k1 = sk[2 * t + 1];
+    x1 = si[2 * t + 1];
+  }
+  for (uint32_t size = 2; size <= np2; size <<= 1)
+    for (uint32_t stride = size >> 1; stride; stride >>= 1) {
+      if (stride == 1) {                                 // elements 2t, 2t+1 of this thread
+        const bool up = ((2 * t) & size) == 0;
+        if (cta_pair_less(k1, x1, k0, x0) == up) {
+          const uint64_t tk = k0;
+          k0 = k1;
+          k1 = tk;
+          const uint32_t tx = x0;
+          x0 = x1;
+          x1 = tx;
+        }
+      } else if (stride < 64) {                          // partner thread t ^ stride/2, same warp
+        const int m = (int)(stride >> 1);
+        const uint64_t p0 = __shfl_xor_sync(0xffffffffu, k0, m), p1 = __shfl_xor_sync(0xffffffffu, k1, m);
+        const uint32_t q0 = __shfl_xor_sync(0xffffffffu, x0, m), q1 = __shfl_xor_sync(0xffffffffu, x1, m);
+        cta_pair_cas(k0, x0, p0, q0, 2 * t, (2 * t) ^ stride, size);
+        cta_pair_cas(k1, x1, p1, q1, 2 * t + 1, (2 * t + 1) ^ stride, size);
+      } else {                                           // through shared memory
+        __syncthreads();
+        if (act) {
+          sk[2 * t] = k0;
+          si[2 * t] = x0;
+          sk[2 * t + 1] = k1;
+          si[2 * t + 1] = x1;
+        }
+        __syncthreads();
+        if (act) {
+          const uint32_t j0 = (2 * t) ^ stride, j1 = (2 * t + 1) ^ stride;
+          const uint64_t p0 = sk[j0], p1 = sk[j1];
+          const uint32_t q0 = si[j0], q1 = si[j1];
+          cta_pair_cas(k0, x0, p0, q0, 2 * t, j0, size);
+          cta_pair_cas(k1, x1, p1, q1, 2 * t + 1, j1, size);
+        }
+      }
+    }
+  __syncthreads();
+  if (act) {
+    sk[2 * t] = k0;
+    si[2 * t] = x0;
+    sk[2 * t + 1] = k1;
+    si[2 * t + 1] = x1;
+  }
+  __syncthreads();
+}
+#endif
 
 // Replayable prefix of one update batch (everything up to its single host read-back) as a
 // CUDA graph: small batches are bound by host launch overhead (~12 launches per insert), a
@@ -139,6 +218,7 @@ struct gpma {
   gp::DevBuf b_lpre, b_wk, b_wv, b_dirty, b_scan, b_hist, b_stage[4], b_misc, b_misc2, b_misc3;
   gp::Ctrl *ctrl_d = nullptr;
   gp::Ctrl *ctrl_h = nullptr;     // pinned mirror
+  uint32_t ctrl_seq = 0;          // sequence number of the last mirrored one-kernel call
   void *pin = nullptr;            // 256 B of pinned host scratch (read-backs of small device state)
   gp::Scratch an[gp::AN_N];       // analytics (read-only on the store)
 

@@ -528,28 +528,14 @@ __global__ void __launch_bounds__(1024) k_small_sort(uint64_t *k0, uint32_t *v0,
                                                      uint32_t n) {
   __shared__ uint64_t sk[SS_MAX];
   __shared__ uint32_t si[SS_MAX];
-  uint32_t np2 = 1;
+  uint32_t np2 = 2;
   while (np2 < n) np2 <<= 1;
   for (uint32_t i = threadIdx.x; i < np2; i += blockDim.x) {
     sk[i] = i < n ? k0[i] : ~0ull;
     si[i] = i;
   }
   __syncthreads();
-  for (uint32_t size = 2; size <= np2; size <<= 1)
-    for (uint32_t stride = size >> 1; stride; stride >>= 1) {
-      for (uint32_t i = threadIdx.x; i < np2; i += blockDim.x) {
-        const uint32_t j = i ^ stride;
-        if (j > i) {
-          const bool up = (i & size) == 0;
-          const bool gt = sk[i] > sk[j] || (sk[i] == sk[j] && si[i] > si[j]);
-          if (gt == up) {
-            uint64_t tk = sk[i]; sk[i] = sk[j]; sk[j] = tk;
-            uint32_t ti = si[i]; si[i] = si[j]; si[j] = ti;
-          }
-        }
-      }
-      __syncthreads();
-    }
+  cta_bitonic_sort(sk, si, np2);           // (key, arrival index): stable
   for (uint32_t i = threadIdx.x; i < n; i += blockDim.x) {
     k1[i] = sk[i];
     v1[i] = v0[si[i]];

@@ -18,6 +18,7 @@
 #include <cooperative_groups.h>
 
 #include <algorithm>
+#include <atomic>
 
 #include "gpma_internal.cuh"
 
@@ -49,13 +50,15 @@ __device__ __forceinline__ uint32_t locate_leaf_rows(const uint64_t *__restrict_
   const uint32_t u = (uint32_t)(k >> 32) - rb;
   const ulonglong2 r = make_ulonglong2(__ldg(ro + u), __ldg(ro + u + 1));
   const uint32_t a = (uint32_t)leaf_div(r.x, L);
-  uint32_t lo = a, hi = min((uint32_t)leaf_div(r.y, L) + 1, nleaves);
+  // the answer is >= a either way, so head[a] is never probed (monotone heads: if head[a] > k
+  // every later head is too and the search ends at a)
+  uint32_t lo = a + 1, hi = min((uint32_t)leaf_div(r.y, L) + 1, nleaves);
   while (lo < hi) {
     uint32_t mid = (lo + hi) >> 1;
     if (__ldg(head + mid) <= k) lo = mid + 1;
     else hi = mid;
   }
-  return lo > a ? lo - 1 : a;
+  return lo - 1;
 }
 
 // Slot of key k in leaf `base` (or -1): the occupied prefix of a leaf is sorted and the empty
@@ -924,269 +927,6 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
   }
 }
 
-// ---- small batches in ONE kernel (n <= SB_MAX): the paper names kernel-call overheads as what
-// dominates small batches (P:1337-1341).  A single CTA validates the batch (nothing changes on
-// an error), sorts it by key in shared memory (bitonic, arrival index breaks ties: stable, R10),
-// locates every key (R9), forms the leaf groups, merges them (leaf_group_merge, leaves staged
-// in shared-memory rows), compacts the rejected keys -- already key-sorted -- into the pending
-// list for level 1 and mirrors its control block to pinned host memory: one launch and one
-// host synchronisation per call instead of a dozen launches.  Lazy deletes likewise.
-constexpr int SB_T = 1024, SB_MAX = 2048, SB_ROWS = 256, SB_DEL_MAX = 4096;
-constexpr size_t SB_ROWK_OFF = ((size_t)SB_MAX * 8 + (size_t)SB_MAX * 4 * 2 + (size_t)(SB_MAX + 1) * 4 * 2 + 15) & ~(size_t)15;
-__host__ __device__ constexpr size_t sb_smem_bytes(int L) { return SB_ROWK_OFF + (size_t)SB_ROWS * (L + 1) * 12; }
-
-__device__ __forceinline__ void sb_block_scan2(uint32_t (&v)[2], uint32_t *wsum, uint32_t *total) {
-  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-  const uint32_t t = v[0] + v[1];
-  uint32_t x = t;
-#pragma unroll
-  for (int o = 1; o < 32; o <<= 1) {
-    const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
-    if (lane >= o) x += y;
-  }
-  if (lane == 31) wsum[warp] = x;
-  __syncthreads();
-  if (warp == 0) {
-    uint32_t w = wsum[lane];
-#pragma unroll
-    for (int o = 1; o < 32; o <<= 1) {
-      const uint32_t y = __shfl_up_sync(0xffffffffu, w, o);
-      if (lane >= o) w += y;
-    }
-    wsum[lane] = w;
-  }
-  __syncthreads();
-  const uint32_t base = (warp ? wsum[warp - 1] : 0) + x - t;
-  *total = wsum[31];
-  __syncthreads();
-  v[1] = base + v[0];
-  v[0] = base;
-}
-
-template <int L>
-__global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
-                                                       uint32_t n, uint64_t *key, uint32_t *val, uint32_t *cnt,
-                                                       uint32_t *tmask, uint64_t *head, uint64_t *row_offset,
-                                                       uint32_t *deg, uint32_t nleaves, uint32_t rb, uint32_t nr,
-                                                       uint32_t V, uint32_t bound, const uint64_t *__restrict__ ro,
-                                                       uint64_t *pk, uint32_t *pv, uint32_t *pt, uint2 *dirty, Ctrl *c,
-                                                       Ctrl *c_host) {
-  extern __shared__ __align__(16) unsigned char sb_smem[];
-  uint64_t *sk = reinterpret_cast<uint64_t *>(sb_smem);           // [SB_MAX] keys (sorted)
-  uint32_t *si = reinterpret_cast<uint32_t *>(sk + SB_MAX);       // [SB_MAX] arrival index -> sorted values
-  uint32_t *st = si + SB_MAX;                                     // [SB_MAX] target leaves
-  uint32_t *kp = st + SB_MAX;                                     // [SB_MAX + 1] keep flags / group starts
-  uint32_t *gs = kp + SB_MAX + 1;                                 // [SB_MAX + 1] group starts
-  uint64_t *rowk = reinterpret_cast<uint64_t *>(sb_smem + SB_ROWK_OFF);   // [SB_ROWS][L + 1]
-  uint32_t *rowv = reinterpret_cast<uint32_t *>(rowk + SB_ROWS * (L + 1));
-  __shared__ uint32_t wsum[32];
-  __shared__ uint32_t s_stats[3];
-  const int tid = threadIdx.x;
-  if (tid == 0) {
-    c->err = 0;
-    c->nunique = 0;
-    c->windows_rewritten = 0;
-    c->ndirty = 0;
-    c->sum = 0;
-    c->sum2 = 0;
-    c->big = 0;
-    s_stats[0] = s_stats[1] = s_stats[2] = 0;
-  }
-  // validate (RESERVED beats RANGE; nothing is mutated on either)
-  uint32_t e = 0;
-  for (uint32_t i = tid; i < n; i += SB_T) {
-    const uint64_t k = ik[i];
-    const uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
-    if (dst == COL_GUARD || iv[i] == VAL_TOMB) e |= 2u;
-    if (src - rb >= nr || dst >= V) e |= 1u;
-  }
-  e = __syncthreads_or(e) ? (__reduce_or_sync(0xffffffffu, e)) : 0u;
-  if (e) atomicOr(&c->err, e);
-  __syncthreads();
-  if (c->err) {
-    if (tid == 0) *c_host = *c;
-    return;
-  }
-  // stable sort by key (bitonic over the next power of two; the arrival index breaks ties)
-  uint32_t np2 = 1;
-  while (np2 < n) np2 <<= 1;
-  for (uint32_t i = tid; i < np2; i += SB_T) {
-    sk[i] = i < n ? ik[i] : KEY_NONE;
-    si[i] = i;
-  }
-  __syncthreads();
-  for (uint32_t size = 2; size <= np2; size <<= 1)
-    for (uint32_t stride = size >> 1; stride; stride >>= 1) {
-      for (uint32_t i = tid; i < np2; i += SB_T) {
-        const uint32_t j = i ^ stride;
-        if (j > i) {
-          const bool up = (i & size) == 0;
-          const bool gt = sk[i] > sk[j] || (sk[i] == sk[j] && si[i] > si[j]);
-          if (gt == up) {
-            const uint64_t tk = sk[i];
-            sk[i] = sk[j];
-            sk[j] = tk;
-            const uint32_t ti = si[i];
-            si[i] = si[j];
-            si[j] = ti;
-          }
-        }
-      }
-      __syncthreads();
-    }
-  // values in key order, targets (R9), group heads
-  uint32_t f[2];
-  for (int q = 0; q < 2; ++q) {
-    const uint32_t i = tid * 2 + q;
-    f[q] = 0;
-    if (i < n) {
-      si[i] = iv[si[i]];
-      st[i] = locate_leaf_rows(head, nleaves, ro, rb, L, sk[i]);
-    }
-  }
-  __syncthreads();
-  for (int q = 0; q < 2; ++q) {
-    const uint32_t i = tid * 2 + q;
-    f[q] = (i < n && (i == 0 || st[i] != st[i - 1])) ? 1u : 0u;
-  }
-  uint32_t fe[2] = {f[0], f[1]}, ng = 0;
-  sb_block_scan2(fe, wsum, &ng);
-  for (int q = 0; q < 2; ++q)
-    if (f[q]) gs[fe[q]] = tid * 2 + q;
-  if (tid == 0) gs[ng] = n;
-  __syncthreads();
-  // the leaf groups, SB_ROWS at a time, each leaf in a shared-memory row
-  const UpdDirect U{sk, si};
-  for (uint32_t g0 = 0; g0 < ng; g0 += SB_ROWS) {
-    const uint32_t gi = g0 + tid;
-    if (tid < SB_ROWS && gi < ng) {
-      const uint32_t j0 = gs[gi], j1 = gs[gi + 1], t = st[j0];
-      const uint64_t lb = (uint64_t)t * L;
-      uint64_t *rk = rowk + tid * (L + 1);
-      uint32_t *rv = rowv + tid * (L + 1);
-      for (int p = 0; p < L; ++p) {
-        rk[p] = key[lb + p];
-        rv[p] = val[lb + p];
-      }
-      const LeafOut o = leaf_group_merge<true>(rk, rv, (uint32_t)L, t, j0, j1, U, bound, kp, key, cnt, tmask, head,
-                                               row_offset, deg, rb, dirty, c);
-      if (o.ok)
-        for (int p = 0; p < L; ++p) key[lb + p] = rk[p];
-      if (o.ok || o.hitm)
-        for (int p = 0; p < L; ++p) val[lb + p] = rv[p];
-      atomicAdd(&s_stats[0], o.ok ? 1u : 0u);
-      atomicAdd(&s_stats[1], o.nnew);
-      atomicAdd(&s_stats[2], o.effs);
-    }
-  }
-  __syncthreads();
-  // the rejected new keys, in key order, with their targets: the pending list of level 1
-  uint32_t kf[2];
-  for (int q = 0; q < 2; ++q) {
-    const uint32_t i = tid * 2 + q;
-    kf[q] = i < n ? kp[i] : 0u;
-  }
-  uint32_t kq[2] = {kf[0], kf[1]}, npend = 0;
-  sb_block_scan2(kq, wsum, &npend);
-  for (int q = 0; q < 2; ++q) {
-    const uint32_t i = tid * 2 + q;
-    if (kf[q]) {
-      pk[kq[q]] = sk[i];
-      pv[kq[q]] = si[i];
-      pt[kq[q]] = st[i];
-    }
-  }
-  __syncthreads();
-  if (tid == 0) {
-    c->windows_rewritten += s_stats[0];
-    c->sum = s_stats[1];              // new keys (pending after the pre-pass, in the old terms)
-    c->nunique = s_stats[2];
-    c->sum2 = npend;                  // pending after level 0
-    __threadfence_system();
-    *c_host = *c;                     // the control block, mirrored (zero-copy) for the host
-  }
-}
-
-// small lazy-delete batch: validate, then mark (P:1260-1266), one CTA, one launch
-__global__ void __launch_bounds__(SB_T) k_small_delete(const uint64_t *__restrict__ ik, uint32_t n,
-                                                       const uint64_t *__restrict__ key, uint32_t *val, uint32_t *cnt,
-                                                       const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
-                                                       uint32_t *tmask, uint32_t *deg, uint32_t rb, uint32_t nr,
-                                                       uint32_t V, const uint64_t *__restrict__ ro, Ctrl *c,
-                                                       Ctrl *c_host) {
-  const int tid = threadIdx.x;
-  if (tid == 0) {
-    c->err = 0;
-    c->nunique = 0;
-    c->sum = 0;
-    c->sum2 = 0;
-  }
-  uint32_t e = 0;
-  for (uint32_t i = tid; i < n; i += SB_T) {
-    const uint64_t k = ik[i];
-    const uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
-    if (dst == COL_GUARD) e |= 2u;
-    if (src - rb >= nr || dst >= V) e |= 1u;
-  }
-  e = __syncthreads_or(e) ? (__reduce_or_sync(0xffffffffu, e)) : 0u;
-  if (e) atomicOr(&c->err, e);
-  __syncthreads();
-  if (!c->err) {
-    for (uint32_t i = tid; i < n; i += SB_T) {
-      const uint64_t k = ik[i];
-      const uint32_t t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
-      const uint64_t base = (uint64_t)t * L;
-      const int p = find_in_leaf(key, base, L, k);
-      if (p < 0) continue;
-      uint32_t old = val[base + p];
-      while (old != VAL_TOMB) {                          // duplicates: one of them accounts it
-        const uint32_t seen = atomicCAS(&val[base + p], old, VAL_TOMB);
-        if (seen == old) {
-          atomicSub(&cnt[t], 1u);
-          atomicOr(&tmask[t], 1u << p);
-          atomicSub(&deg[(uint32_t)(k >> 32) - rb], 1u);
-          break;
-        }
-        old = seen;
-      }
-    }
-  }
-  __syncthreads();
-  if (tid == 0) {
-    __threadfence_system();
-    *c_host = *c;
-  }
-}
-
-// the rejected new keys (keep[j] = 1) of the leaf-sorted batch, compacted in leaf order with
-// their targets, plus 0..p-1 (the sort of the pending keys permutes it)
-__global__ void k_pend_gather(const uint32_t *__restrict__ keep, const uint32_t *__restrict__ pos, uint64_t n,
-                              const uint32_t *__restrict__ tix, const uint64_t *__restrict__ tk,
-                              const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
-                              uint64_t *__restrict__ pk, uint32_t *__restrict__ pv, uint32_t *__restrict__ pt,
-                              uint32_t *__restrict__ seq) {
-  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < n;
-       j += (uint64_t)gridDim.x * blockDim.x) {
-    if (!keep[j]) continue;
-    const uint32_t d = pos[j], i = tix[j];
-    pk[d] = ik[i];
-    pv[d] = iv[i];
-    pt[d] = (uint32_t)tk[j];
-    seq[d] = d;
-  }
-}
-
-// pending list in key order: values and targets follow the sort's permutation
-__global__ void k_pend_permute(const uint32_t *__restrict__ perm, uint64_t p, const uint32_t *__restrict__ pv_in,
-                               const uint32_t *__restrict__ pt_in, uint32_t *__restrict__ pv, uint32_t *__restrict__ pt) {
-  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < p;
-       j += (uint64_t)gridDim.x * blockDim.x) {
-    const uint32_t q = perm[j];
-    pv[j] = pv_in[q];
-    pt[j] = pt_in[q];
-  }
-}
-
 // ---- R-way interleaved locate (memory-level parallelism): the random loads of R independent
 // keys -- row offsets, head probes, the first 8 slots of the target leaf -- are issued together,
 // so a thread keeps R dependent chains in flight instead of one (the kernels below are bound by
@@ -1209,8 +949,10 @@ __device__ __forceinline__ void locate_leaf_rows_r(const uint64_t *__restrict__ 
   }
 #pragma unroll
   for (int q = 0; q < R; ++q) {
+    // the answer is >= a either way (see locate_leaf_rows), so the search starts past a: one
+    // random probe less per key, none for a row inside one leaf
     a[q] = (uint32_t)leaf_div(r[q].x, L);
-    lo[q] = a[q];
+    lo[q] = a[q] + 1;
     hi[q] = v[q] ? min((uint32_t)leaf_div(r[q].y, L) + 1, nleaves) : a[q];
   }
   bool any = true;
@@ -1232,7 +974,7 @@ __device__ __forceinline__ void locate_leaf_rows_r(const uint64_t *__restrict__ 
       }
   }
 #pragma unroll
-  for (int q = 0; q < R; ++q) t[q] = lo[q] > a[q] ? lo[q] - 1 : a[q];
+  for (int q = 0; q < R; ++q) t[q] = v[q] ? lo[q] - 1 : a[q];
 }
 
 // slot of k[q] in its leaf t[q] (or -1) for R keys: the leaves' slots fetched 8 at a time, the
@@ -1273,8 +1015,309 @@ __device__ __forceinline__ void find_in_leaf_r(const uint64_t *__restrict__ key,
   }
 }
 
+// The control block mirrored into pinned host memory by the kernel's thread 0 (after a barrier):
+// the fields, a system fence, then the sequence number -- the host sees the whole block once it
+// sees the number (wait_ctrl), without waiting for the kernel's completion to reach the stream.
+__device__ __forceinline__ void mirror_ctrl(const Ctrl *c, Ctrl *c_host, uint32_t seq) {
+  __threadfence_system();
+  *c_host = *c;
+  __threadfence_system();
+  *reinterpret_cast<volatile uint32_t *>(&c_host->seq) = seq;
+}
+
+// ---- small batches in ONE kernel (n <= SB_MAX): the paper names kernel-call overheads as what
+// dominates small batches (P:1337-1341).  A single CTA validates the batch (nothing changes on
+// an error), sorts it by key in shared memory (bitonic, arrival index breaks ties: stable, R10),
+// locates every key (R9), forms the leaf groups, merges them (leaf_group_merge, leaves staged
+// in shared-memory rows), compacts the rejected keys -- already key-sorted -- into the pending
+// list for level 1 and mirrors its control block to pinned host memory: one launch and one
+// host synchronisation per call instead of a dozen launches.  Lazy deletes likewise.
+constexpr int SB_T = 1024, SB_MAX = 2048, SB_ROWS = 512, SB_DEL_MAX = 4096;
+constexpr size_t SB_ROWK_OFF = ((size_t)SB_MAX * 8 + (size_t)SB_MAX * 4 * 2 + (size_t)(SB_MAX + 1) * 4 * 2 + 15) & ~(size_t)15;
+__host__ __device__ constexpr size_t sb_smem_bytes(int L) { return SB_ROWK_OFF + (size_t)SB_ROWS * (L + 1) * 12; }
+
+__device__ __forceinline__ void sb_block_scan2(uint32_t (&v)[2], uint32_t *wsum, uint32_t *total) {
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint32_t t = v[0] + v[1];
+  uint32_t x = t;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if (lane >= o) x += y;
+  }
+  if (lane == 31) wsum[warp] = x;
+  __syncthreads();
+  if (warp == 0) {
+    uint32_t w = wsum[lane];
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, w, o);
+      if (lane >= o) w += y;
+    }
+    wsum[lane] = w;
+  }
+  __syncthreads();
+  const uint32_t base = (warp ? wsum[warp - 1] : 0) + x - t;
+  *total = wsum[31];
+  __syncthreads();
+  v[1] = base + v[0];
+  v[0] = base;
+}
+
+template <int L>
+__global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
+                                                       uint32_t n, uint64_t *key, uint32_t *val, uint32_t *cnt,
+                                                       uint32_t *tmask, uint64_t *head, uint64_t *row_offset,
+                                                       uint32_t *deg, uint32_t nleaves, uint32_t rb, uint32_t nr,
+                                                       uint32_t V, uint32_t bound, const uint64_t *__restrict__ ro,
+                                                       uint64_t *pk, uint32_t *pv, uint32_t *pt, uint2 *dirty, Ctrl *c,
+                                                       Ctrl *c_host, uint32_t seq) {
+  extern __shared__ __align__(16) unsigned char sb_smem[];
+  uint64_t *sk = reinterpret_cast<uint64_t *>(sb_smem);           // [SB_MAX] keys (sorted)
+  uint32_t *si = reinterpret_cast<uint32_t *>(sk + SB_MAX);       // [SB_MAX] arrival index -> sorted values
+  uint32_t *st = si + SB_MAX;                                     // [SB_MAX] target leaves
+  uint32_t *kp = st + SB_MAX;                                     // [SB_MAX + 1] keep flags / group starts
+  uint32_t *gs = kp + SB_MAX + 1;                                 // [SB_MAX + 1] group starts
+  uint64_t *rowk = reinterpret_cast<uint64_t *>(sb_smem + SB_ROWK_OFF);   // [SB_ROWS][L + 1]
+  uint32_t *rowv = reinterpret_cast<uint32_t *>(rowk + SB_ROWS * (L + 1));
+  __shared__ uint32_t wsum[32];
+  __shared__ uint32_t s_stats[3];
+  const int tid = threadIdx.x;
+  if (tid == 0) {
+    c->err = 0;
+    c->nunique = 0;
+    c->windows_rewritten = 0;
+    c->ndirty = 0;
+    c->sum = 0;
+    c->sum2 = 0;
+    c->big = 0;
+    s_stats[0] = s_stats[1] = s_stats[2] = 0;
+  }
+  // load + validate (RESERVED beats RANGE; nothing is mutated on either) + locate (R9): each
+  // thread's two keys located together while the batch is still in arrival order (an invalid
+  // key is not located); values and targets parked by arrival index in kp / gs
+  uint32_t e = 0;
+  {
+    uint64_t k[2];
+    bool v[2];
+    for (int q = 0; q < 2; ++q) {
+      const uint32_t i = tid + q * SB_T;
+      v[q] = i < n;
+      k[q] = v[q] ? ik[i] : 0ull;
+      const uint32_t x = v[q] ? iv[i] : 0u;
+      if (v[q]) {
+        const uint32_t src = (uint32_t)(k[q] >> 32), dst = (uint32_t)k[q];
+        uint32_t ee = 0;
+        if (dst == COL_GUARD || x == VAL_TOMB) ee |= 2u;
+        if (src - rb >= nr || dst >= V) ee |= 1u;
+        e |= ee;
+        v[q] = ee == 0;
+        sk[i] = k[q];
+        si[i] = i;
+        kp[i] = x;
+      }
+    }
+    uint32_t t[2];
+    locate_leaf_rows_r<2>(head, nleaves, ro, rb, L, k, v, t);
+    for (int q = 0; q < 2; ++q) {
+      const uint32_t i = tid + q * SB_T;
+      if (i < n) gs[i] = t[q];
+    }
+  }
+  e = __syncthreads_or(e) ? (__reduce_or_sync(0xffffffffu, e)) : 0u;
+  if (e) atomicOr(&c->err, e);
+  __syncthreads();
+  if (c->err) {
+    if (tid == 0) mirror_ctrl(c, c_host, seq);
+    return;
+  }
+  // stable sort by key (the arrival index breaks ties), padding up to a power of two
+  uint32_t np2 = 2;
+  while (np2 < n) np2 <<= 1;
+  for (uint32_t i = n + tid; i < np2; i += SB_T) {
+    sk[i] = KEY_NONE;
+    si[i] = i;
+  }
+  __syncthreads();
+  cta_bitonic_sort(sk, si, np2);
+  // values and targets in key order, group heads
+  uint32_t f[2], sv_[2], st_[2];
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    if (i < n) {
+      sv_[q] = kp[si[i]];
+      st_[q] = gs[si[i]];
+    }
+  }
+  __syncthreads();
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    if (i < n) {
+      si[i] = sv_[q];
+      st[i] = st_[q];
+    }
+  }
+  __syncthreads();
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    f[q] = (i < n && (i == 0 || st[i] != st[i - 1])) ? 1u : 0u;
+  }
+  uint32_t fe[2] = {f[0], f[1]}, ng = 0;
+  sb_block_scan2(fe, wsum, &ng);
+  for (int q = 0; q < 2; ++q)
+    if (f[q]) gs[fe[q]] = tid * 2 + q;
+  if (tid == 0) gs[ng] = n;
+  __syncthreads();
+  // the leaf groups, SB_ROWS at a time, each leaf in a shared-memory row
+  const UpdDirect U{sk, si};
+  uint32_t a_ok = 0, a_new = 0, a_effs = 0;
+  for (uint32_t g0 = 0; g0 < ng; g0 += SB_ROWS) {
+    const uint32_t gi = g0 + tid;
+    if (tid < SB_ROWS && gi < ng) {
+      const uint32_t j0 = gs[gi], j1 = gs[gi + 1], t = st[j0];
+      const uint64_t lb = (uint64_t)t * L;
+      uint64_t *rk = rowk + tid * (L + 1);
+      uint32_t *rv = rowv + tid * (L + 1);
+      // the leaf's L keys and values in flight together (16-B loads into registers, then the
+      // row): loads interleaved with the shared-memory stores through the generic pointers
+      // were serialised one DRAM round trip per slot
+      ulonglong2 lk[L / 2];
+      uint4 lv[L / 4];
+#pragma unroll
+      for (int p = 0; p < L / 2; ++p) lk[p] = __ldcg(reinterpret_cast<const ulonglong2 *>(key + lb) + p);
+#pragma unroll
+      for (int p = 0; p < L / 4; ++p) lv[p] = __ldcg(reinterpret_cast<const uint4 *>(val + lb) + p);
+#pragma unroll
+      for (int p = 0; p < L / 2; ++p) {
+        rk[2 * p] = lk[p].x;
+        rk[2 * p + 1] = lk[p].y;
+      }
+#pragma unroll
+      for (int p = 0; p < L / 4; ++p) {
+        rv[4 * p] = lv[p].x;
+        rv[4 * p + 1] = lv[p].y;
+        rv[4 * p + 2] = lv[p].z;
+        rv[4 * p + 3] = lv[p].w;
+      }
+      const LeafOut o = leaf_group_merge<true>(rk, rv, (uint32_t)L, t, j0, j1, U, bound, kp, key, cnt, tmask, head,
+                                               row_offset, deg, rb, dirty, c);
+      if (o.ok)
+        for (int p = 0; p < L; ++p) key[lb + p] = rk[p];
+      if (o.ok || o.hitm)
+        for (int p = 0; p < L; ++p) val[lb + p] = rv[p];
+      a_ok += o.ok ? 1u : 0u;
+      a_new += o.nnew;
+      a_effs += o.effs;
+    }
+  }
+  a_ok = __reduce_add_sync(0xffffffffu, a_ok);         // one shared atomic per warp
+  a_new = __reduce_add_sync(0xffffffffu, a_new);
+  a_effs = __reduce_add_sync(0xffffffffu, a_effs);
+  if ((tid & 31) == 0 && (a_ok | a_new | a_effs)) {
+    atomicAdd(&s_stats[0], a_ok);
+    atomicAdd(&s_stats[1], a_new);
+    atomicAdd(&s_stats[2], a_effs);
+  }
+  __syncthreads();
+  // the rejected new keys, in key order, with their targets: the pending list of level 1
+  uint32_t kf[2];
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    kf[q] = i < n ? kp[i] : 0u;
+  }
+  uint32_t kq[2] = {kf[0], kf[1]}, npend = 0;
+  sb_block_scan2(kq, wsum, &npend);
+  for (int q = 0; q < 2; ++q) {
+    const uint32_t i = tid * 2 + q;
+    if (kf[q]) {
+      pk[kq[q]] = sk[i];
+      pv[kq[q]] = si[i];
+      pt[kq[q]] = st[i];
+    }
+  }
+  __syncthreads();
+  if (tid == 0) {
+    c->windows_rewritten += s_stats[0];
+    c->sum = s_stats[1];              // new keys (pending after the pre-pass, in the old terms)
+    c->nunique = s_stats[2];
+    c->sum2 = npend;                  // pending after level 0
+    mirror_ctrl(c, c_host, seq);      // the control block, mirrored (zero-copy) for the host
+  }
+}
+
+// small lazy-delete batch: validate, then mark (P:1260-1266), one CTA, one launch
+__global__ void __launch_bounds__(SB_T) k_small_delete(const uint64_t *__restrict__ ik, uint32_t n,
+                                                       const uint64_t *__restrict__ key, uint32_t *val, uint32_t *cnt,
+                                                       const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
+                                                       uint32_t *tmask, uint32_t *deg, uint32_t rb, uint32_t nr,
+                                                       uint32_t V, const uint64_t *__restrict__ ro, Ctrl *c,
+                                                       Ctrl *c_host, uint32_t seq) {
+  const int tid = threadIdx.x;
+  if (tid == 0) {
+    c->err = 0;
+    c->nunique = 0;
+    c->sum = 0;
+    c->sum2 = 0;
+  }
+  uint32_t e = 0;
+  for (uint32_t i = tid; i < n; i += SB_T) {
+    const uint64_t k = ik[i];
+    const uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
+    if (dst == COL_GUARD) e |= 2u;
+    if (src - rb >= nr || dst >= V) e |= 1u;
+  }
+  e = __syncthreads_or(e) ? (__reduce_or_sync(0xffffffffu, e)) : 0u;
+  if (e) atomicOr(&c->err, e);
+  __syncthreads();
+  if (!c->err) {
+    for (uint32_t i = tid; i < n; i += SB_T) {
+      const uint64_t k = ik[i];
+      const uint32_t t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
+      const uint64_t base = (uint64_t)t * L;
+      const int p = find_in_leaf(key, base, L, k);
+      if (p < 0) continue;
+      if (atomicExch(&val[base + p], VAL_TOMB) != VAL_TOMB) {   // duplicates: one of them accounts it
+        atomicSub(&cnt[t], 1u);
+        atomicOr(&tmask[t], 1u << p);
+        atomicSub(&deg[(uint32_t)(k >> 32) - rb], 1u);
+      }
+    }
+  }
+  __syncthreads();
+  if (tid == 0) mirror_ctrl(c, c_host, seq);
+}
+
+// the rejected new keys (keep[j] = 1) of the leaf-sorted batch, compacted in leaf order with
+// their targets, plus 0..p-1 (the sort of the pending keys permutes it)
+__global__ void k_pend_gather(const uint32_t *__restrict__ keep, const uint32_t *__restrict__ pos, uint64_t n,
+                              const uint32_t *__restrict__ tix, const uint64_t *__restrict__ tk,
+                              const uint64_t *__restrict__ ik, const uint32_t *__restrict__ iv,
+                              uint64_t *__restrict__ pk, uint32_t *__restrict__ pv, uint32_t *__restrict__ pt,
+                              uint32_t *__restrict__ seq) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < n;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    if (!keep[j]) continue;
+    const uint32_t d = pos[j], i = tix[j];
+    pk[d] = ik[i];
+    pv[d] = iv[i];
+    pt[d] = (uint32_t)tk[j];
+    seq[d] = d;
+  }
+}
+
+// pending list in key order: values and targets follow the sort's permutation
+__global__ void k_pend_permute(const uint32_t *__restrict__ perm, uint64_t p, const uint32_t *__restrict__ pv_in,
+                               const uint32_t *__restrict__ pt_in, uint32_t *__restrict__ pv, uint32_t *__restrict__ pt) {
+  for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < p;
+       j += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t q = perm[j];
+    pv[j] = pv_in[q];
+    pt[j] = pt_in[q];
+  }
+}
+
 // Lazy deletion (R12) in arrival order, R keys per thread interleaved.  Duplicates
-// race on the same slot; the CAS on the value lets exactly one account the deletion.
+// race on the same slot; the exchange on the value lets exactly one account the deletion.
 template <int LD_R>
 __global__ void __launch_bounds__(256) k_lazy_delete_r(const uint64_t *__restrict__ keys, uint64_t n,
                                                        const uint64_t *__restrict__ key, uint32_t *val,
@@ -1297,23 +1340,19 @@ __global__ void __launch_bounds__(256) k_lazy_delete_r(const uint64_t *__restric
     locate_leaf_rows_r<LD_R>(head, nleaves, ro, rb, L, k, v, t);
     int p[LD_R];
     find_in_leaf_r<LD_R>(key, L, k, v, t, p);
+    // one exchange per found key: the copy that swaps a live value for TOMB accounts it
+    // (a duplicate, or an already-tombstoned slot, reads TOMB back)
     uint32_t old[LD_R];
 #pragma unroll
-    for (int q = 0; q < LD_R; ++q) old[q] = p[q] >= 0 ? val[(uint64_t)t[q] * L + p[q]] : VAL_TOMB;
+    for (int q = 0; q < LD_R; ++q)
+      old[q] = p[q] >= 0 ? atomicExch(&val[(uint64_t)t[q] * L + p[q]], VAL_TOMB) : VAL_TOMB;
 #pragma unroll
-    for (int q = 0; q < LD_R; ++q) {
-      const uint64_t s = (uint64_t)t[q] * L + (p[q] >= 0 ? p[q] : 0);
-      while (old[q] != VAL_TOMB) {
-        const uint32_t seen = atomicCAS(&val[s], old[q], VAL_TOMB);
-        if (seen == old[q]) {
-          atomicSub(&cnt[t[q]], 1u);
-          atomicOr(&tmask[t[q]], 1u << p[q]);
-          atomicSub(&deg[(uint32_t)(k[q] >> 32) - rb], 1u);
-          break;
-        }
-        old[q] = seen;
+    for (int q = 0; q < LD_R; ++q)
+      if (old[q] != VAL_TOMB) {
+        atomicSub(&cnt[t[q]], 1u);
+        atomicOr(&tmask[t[q]], 1u << p[q]);
+        atomicSub(&deg[(uint32_t)(k[q] >> 32) - rb], 1u);
       }
-    }
   }
 }
 
@@ -3784,12 +3823,42 @@ static bool small_batch_path(gpma *g, uint64_t n, int op, int path) {
   return false;
 }
 
+static uint32_t next_seq(gpma *g) {
+  if (++g->ctrl_seq == 0) g->ctrl_seq = 1;            // 0: what the mirror copies before the number
+  return g->ctrl_seq;
+}
+
+// Wait for the one-kernel call's control block: spin on its sequence number in pinned memory
+// (GPMA_SPIN=0: cudaStreamSynchronize).  The stream is polled now and then, so a failed kernel
+// (which never writes the number) surfaces its error instead of hanging the host.
+static cudaError_t wait_ctrl(gpma *g, cudaStream_t s) {
+  static const bool spin = [] {
+    const char *e = getenv("GPMA_SPIN");
+    return !e || atoi(e) != 0;
+  }();
+  if (spin) {
+    const volatile uint32_t *q = &g->ctrl_h->seq;
+    for (uint64_t it = 1;; ++it) {
+      if (*q == g->ctrl_seq) {
+        std::atomic_thread_fence(std::memory_order_acquire);
+        return cudaSuccess;
+      }
+      if ((it & 4095) == 0) {
+        const cudaError_t e = cudaStreamQuery(s);
+        if (e == cudaSuccess) break;                     // done without the number: let sync decide
+        if (e != cudaErrorNotReady) return e;
+      }
+    }
+  }
+  return cudaStreamSynchronize(s);
+}
+
 static gpma_status run_small(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, int op, cudaStream_t s) {
   const uint64_t nl = g->cap / g->L;
   const uint64_t *ro = g->rows_indexed ? g->row_offset : nullptr;
   if (op == GPMA_DELETE) {
     GP_LAUNCH(g, k_small_delete, 1, SB_T, 0, s, ik, (uint32_t)n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
-              tmask_of(g), g->deg, g->rb, g->nr, g->V, ro, g->ctrl_d, g->ctrl_h);
+              tmask_of(g), g->deg, g->rb, g->nr, g->V, ro, g->ctrl_d, g->ctrl_h, next_seq(g));
     GP_CHECK(g, cudaGetLastError());
     return GPMA_OK;
   }
@@ -3809,7 +3878,8 @@ static gpma_status run_small(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, in
 #define GP_SMALL_INS(LL)                                                                                         \
   GP_LAUNCH(g, k_small_insert<LL>, 1, SB_T, sb_smem_bytes(LL), s, ik, iv, (uint32_t)n, g->key, g->val, g->cnt,   \
             tmask_of(g), g->head, g->row_offset, g->deg, (uint32_t)nl, g->rb, g->nr, g->V, bound, ro, pk, pv, pt, \
-            dirty, g->ctrl_d, g->ctrl_h)
+            dirty, g->ctrl_d, g->ctrl_h, seq)
+  const uint32_t seq = next_seq(g);
   if (g->L == 16) GP_SMALL_INS(16);
   else if (g->L == 8) GP_SMALL_INS(8);
   else GP_SMALL_INS(4);
@@ -3942,7 +4012,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
     // the one-kernel small batch only reads the batch: no staging copy of a device batch
     if ((st = run_small(g, const_cast<uint64_t *>(keys), const_cast<uint32_t *>(vals), n, op, s))) return st;
     path = path == PATH_INS_LEAF || path == PATH_INS_FUSED ? PATH_INS_SMALL : path;
-    GP_CHECK(g, cudaStreamSynchronize(s));
+    GP_CHECK(g, wait_ctrl(g, s));
     if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) {
       g->last.last_unique = n;
       return status_of(g);
@@ -3955,13 +4025,14 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   uint32_t *iv = (uint32_t *)g->b_stage[1].p;
   GP_CHECK(g, stage_in(g, ik, keys, n * 8, s));
   if (op == GPMA_INSERT) GP_CHECK(g, stage_in(g, iv, vals, n * 4, s));
-  if (small_batch_path(g, n, op, path)) {
+  const bool small = small_batch_path(g, n, op, path);
+  if (small) {
     if ((st = run_small(g, ik, iv, n, op, s))) return st;
     path = path == PATH_INS_LEAF || path == PATH_INS_FUSED ? PATH_INS_SMALL : path;
   } else if ((st = run_prefix(g, ik, iv, n, op, &srt, s))) {
     return st;
   }
-  GP_CHECK(g, cudaStreamSynchronize(s));             // the one host round trip of the batch
+  GP_CHECK(g, small ? wait_ctrl(g, s) : cudaStreamSynchronize(s));   // the one host round trip of the batch
   if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) {
     g->last.last_unique = n;   // (lazy deletes are idempotent; the sorted path marks each key once)
     return status_of(g);

@@ -178,18 +178,66 @@ def _check_arr(a, itemsize: int, min_numel: int, what: str, device=None):
         raise ValueError(f"{what}: tensor on cuda:{dev.index}, handle on cuda:{device}")
 
 
-def _stream(stream):
-    if stream is None:
+_torch = None
+_raw_stream = None
+
+
+def _torch_mod():
+    """torch (imported once) and its raw current-stream getter, or None without CUDA."""
+    global _torch, _raw_stream
+    if _torch is None:
         try:
             import torch
+            _torch = torch
             if torch.cuda.is_available():
-                return torch.cuda.current_stream().cuda_stream or None
+                _raw_stream = getattr(torch._C, "_cuda_getCurrentRawStream", None) or (
+                    lambda d: torch.cuda.current_stream(d).cuda_stream)
         except Exception:
-            pass
-        return None
+            _torch = False
+    return _torch
+
+
+def _stream(stream, device=None):
+    if stream is None:
+        _torch_mod()
+        if _raw_stream is None:
+            return None
+        if device is None:
+            device = _torch.cuda.current_device()
+        return _raw_stream(device) or None
     if isinstance(stream, int):
         return stream or None
     return stream.cuda_stream or None
+
+
+def _targ(a, itemsize: int, min_numel: int, what: str, device):
+    """(pointer, numel) of an update / result array with _check_arr's checks, fast path for torch
+    tensors (the per-call binding cost of the small-batch update path)."""
+    if a is None:
+        return None, 0
+    T = _torch_mod()
+    if T and type(a) is T.Tensor:
+        n = a.numel()
+        if a.element_size() != itemsize:
+            raise ValueError(f"{what}: element size {a.element_size()} B, expected {itemsize} B")
+        if n < min_numel:
+            raise ValueError(f"{what}: {n} elements, need at least {min_numel}")
+        if a.is_cuda and device is not None and a.get_device() != device:
+            raise ValueError(f"{what}: tensor on cuda:{a.get_device()}, handle on cuda:{device}")
+        if not a.is_contiguous():
+            raise ValueError("array must be contiguous")
+        return a.data_ptr() or None, n
+    _check_arr(a, itemsize, min_numel, what, device)
+    return _ptr(a), _numel(a)
+    if isinstance(stream, int):
+        return stream or None
+    return stream.cuda_stream or None
+
+
+def _update(*args):
+    global _update
+    _update = lib().gpma_update_batch       # bound once: the ctypes function itself
+    return _update(*args)
 
 
 class Gpma:
@@ -269,10 +317,10 @@ class Gpma:
 
     # -- update -----------------------------------------------------------
     def gpma_update_batch(self, keys, vals=None, op: int = INSERT, stream=None, check: bool = True) -> int:
-        _check_arr(keys, 8, 0, "keys", self.device)
-        _check_arr(vals, 4, _numel(keys), "vals", self.device)
-        st = lib().gpma_update_batch(self._h, _ptr(keys), _ptr(vals), _numel(keys), op, _stream(stream))
-        if check:
+        kp, n = _targ(keys, 8, 0, "keys", self.device)
+        vp, _ = _targ(vals, 4, n, "vals", self.device)
+        st = _update(self._h, kp, vp, n, op, _stream(stream, self.device))
+        if check and st != OK:
             self._check(st, "gpma_update_batch")
         return st
 

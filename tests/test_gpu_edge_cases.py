@@ -127,6 +127,25 @@ def test_sort_tiles_and_stability(n):
     assert_same_csr(g, o)
 
 
+@pytest.mark.parametrize("n", [1, 2, 3, 31, 33, 63, 64, 65, 127, 129, 1000, 1025, 2047, 2048])
+def test_small_path_sizes_and_stability(n, monkeypatch):
+    """The one-kernel small-batch insert (GPMA_SMALL=2048: every size here) across the bitonic
+    sort's register / shuffle / shared-memory stride regimes and padding, with duplicated keys
+    (the LAST copy wins, R10) into a populated store, then the same keys deleted."""
+    monkeypatch.setenv("GPMA_SMALL", "2048")
+    rng = np.random.default_rng(77 + n)
+    V = 1 << 10
+    k0 = np.unique(rng.integers(0, V, 3000) << 32 | rng.integers(0, V, 3000)).astype(np.uint64).tolist()
+    g, o = _pair(V, k0, [1] * len(k0))
+    pool = np.unique(rng.integers(0, V, 4 * n) << 32 | rng.integers(0, V, 4 * n))[: max(n // 2, 1)]
+    keys = pool[rng.integers(0, pool.size, n)].astype(np.uint64).tolist()
+    vals = rng.integers(0, 1 << 31, n).tolist()
+    _apply(g, o, keys, vals)
+    assert_same_csr(g, o)
+    _apply(g, o, keys[: max(n // 2, 1)], op=1)
+    assert_same_csr(g, o)
+
+
 def test_torch_allocator_hooks():
     """gpma_config.alloc/free through PyTorch's caching allocator (SURVEY §8(b) "Ownership"): the
     store lives in torch's pool while the handle lives, the results are unchanged, and destroy
