@@ -112,6 +112,7 @@ __device__ __forceinline__ void cta_pair_cas(uint64_t &k, uint32_t &x, uint64_t 
 __device__ inline void cta_bitonic_sort(uint64_t *sk, uint32_t *si, uint32_t np2) {
   const uint32_t t = threadIdx.x;
   const bool act = 2 * t < np2;
+  const bool wact = 64 * (t >> 5) < np2;                 // warp-uniform: the warp holds elements
   uint64_t k0 = ~0ull, k1 = ~0ull;
   uint32_t x0 = ~0u, x1 = ~0u;
   if (act) {
@@ -122,6 +123,7 @@ __device__ inline void cta_bitonic_sort(uint64_t *sk, uint32_t *si, uint32_t np2
   }
   for (uint32_t size = 2; size <= np2; size <<= 1)
     for (uint32_t stride = size >> 1; stride; stride >>= 1) {
+      if (stride < 64 && !wact) continue;               // (no barrier below 64)
       if (stride == 1) {                                 // elements 2t, 2t+1 of this thread
         const bool up = ((2 * t) & size) == 0;
         if (cta_pair_less(k1, x1, k0, x0) == up) {
@@ -162,6 +164,59 @@ __device__ inline void cta_bitonic_sort(uint64_t *sk, uint32_t *si, uint32_t np2
     si[2 * t] = x0;
     sk[2 * t + 1] = k1;
     si[2 * t + 1] = x1;
+  }
+  __syncthreads();
+}
+
+// The same network over distinct u64 keys only (sk[0, np2)): one compare and one 64-bit shuffle
+// per element and stage -- for keys that carry their own tie-break (a packed arrival index).
+__device__ inline void cta_bitonic_sort_u64(uint64_t *sk, uint32_t np2) {
+  const uint32_t t = threadIdx.x;
+  const bool act = 2 * t < np2;
+  const bool wact = 64 * (t >> 5) < np2;
+  uint64_t k0 = ~0ull, k1 = ~0ull;
+  if (act) {
+    k0 = sk[2 * t];
+    k1 = sk[2 * t + 1];
+  }
+  for (uint32_t size = 2; size <= np2; size <<= 1)
+    for (uint32_t stride = size >> 1; stride; stride >>= 1) {
+      if (stride < 64 && !wact) continue;
+      if (stride == 1) {
+        const bool up = ((2 * t) & size) == 0;
+        if ((k1 < k0) == up) {
+          const uint64_t tk = k0;
+          k0 = k1;
+          k1 = tk;
+        }
+      } else if (stride < 64) {
+        const int m = (int)(stride >> 1);
+        const uint64_t p0 = __shfl_xor_sync(0xffffffffu, k0, m), p1 = __shfl_xor_sync(0xffffffffu, k1, m);
+        const bool up = ((2 * t) & size) == 0;           // same for 2t and 2t+1 (size >= 4 here)
+        const bool lo = ((2 * t) & stride) == 0;         // this thread holds the lower index of the pair
+        const bool keep_min = lo == up;
+        k0 = keep_min ? min(k0, p0) : max(k0, p0);
+        k1 = keep_min ? min(k1, p1) : max(k1, p1);
+      } else {
+        __syncthreads();
+        if (act) {
+          sk[2 * t] = k0;
+          sk[2 * t + 1] = k1;
+        }
+        __syncthreads();
+        if (act) {
+          const uint64_t p0 = sk[(2 * t) ^ stride], p1 = sk[(2 * t + 1) ^ stride];
+          const bool up = ((2 * t) & size) == 0;
+          const bool keep_min = (((2 * t) & stride) == 0) == up;
+          k0 = keep_min ? min(k0, p0) : max(k0, p0);
+          k1 = keep_min ? min(k1, p1) : max(k1, p1);
+        }
+      }
+    }
+  __syncthreads();
+  if (act) {
+    sk[2 * t] = k0;
+    sk[2 * t + 1] = k1;
   }
   __syncthreads();
 }

@@ -1033,6 +1033,7 @@ __device__ __forceinline__ void mirror_ctrl(const Ctrl *c, Ctrl *c_host, uint32_
 // list for level 1 and mirrors its control block to pinned host memory: one launch and one
 // host synchronisation per call instead of a dozen launches.  Lazy deletes likewise.
 constexpr int SB_T = 1024, SB_MAX = 2048, SB_ROWS = 512, SB_DEL_MAX = 4096;
+constexpr uint64_t SB_DEFAULT = 1024;  // default GPMA_SMALL: inserts and lazy deletes <= it take one kernel
 constexpr size_t SB_ROWK_OFF = ((size_t)SB_MAX * 8 + (size_t)SB_MAX * 4 * 2 + (size_t)(SB_MAX + 1) * 4 * 2 + 15) & ~(size_t)15;
 __host__ __device__ constexpr size_t sb_smem_bytes(int L) { return SB_ROWK_OFF + (size_t)SB_ROWS * (L + 1) * 12; }
 
@@ -1071,7 +1072,7 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
                                                        uint32_t *deg, uint32_t nleaves, uint32_t rb, uint32_t nr,
                                                        uint32_t V, uint32_t bound, const uint64_t *__restrict__ ro,
                                                        uint64_t *pk, uint32_t *pv, uint32_t *pt, uint2 *dirty, Ctrl *c,
-                                                       Ctrl *c_host, uint32_t seq) {
+                                                       Ctrl *c_host, uint32_t seq, uint32_t pbd) {
   extern __shared__ __align__(16) unsigned char sb_smem[];
   uint64_t *sk = reinterpret_cast<uint64_t *>(sb_smem);           // [SB_MAX] keys (sorted)
   uint32_t *si = reinterpret_cast<uint32_t *>(sk + SB_MAX);       // [SB_MAX] arrival index -> sorted values
@@ -1134,12 +1135,27 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
   // stable sort by key (the arrival index breaks ties), padding up to a power of two
   uint32_t np2 = 2;
   while (np2 < n) np2 <<= 1;
-  for (uint32_t i = n + tid; i < np2; i += SB_T) {
-    sk[i] = KEY_NONE;
-    si[i] = i;
+  if (pbd) {
+    // (src - rb, dst, arrival) packed into one distinct u64 (pbd = dst bits; the host checks
+    // that row bits + pbd + 11 <= 64): half the shuffles and one compare per stage
+    for (uint32_t i = tid; i < np2; i += SB_T)
+      sk[i] = i < n ? ((((sk[i] >> 32) - rb) << (pbd + 11)) | ((sk[i] & 0xFFFFFFFFull) << 11) | i) : ~0ull;
+    __syncthreads();
+    cta_bitonic_sort_u64(sk, np2);
+    for (uint32_t i = tid; i < n; i += SB_T) {
+      const uint64_t pw = sk[i];
+      si[i] = (uint32_t)(pw & (SB_MAX - 1));
+      sk[i] = (((pw >> (pbd + 11)) + rb) << 32) | ((pw >> 11) & ((1ull << pbd) - 1));
+    }
+    __syncthreads();
+  } else {
+    for (uint32_t i = n + tid; i < np2; i += SB_T) {
+      sk[i] = KEY_NONE;
+      si[i] = i;
+    }
+    __syncthreads();
+    cta_bitonic_sort(sk, si, np2);
   }
-  __syncthreads();
-  cta_bitonic_sort(sk, si, np2);
   // values and targets in key order, group heads
   uint32_t f[2], sv_[2], st_[2];
   for (int q = 0; q < 2; ++q) {
@@ -1171,40 +1187,82 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
   // the leaf groups, SB_ROWS at a time, each leaf in a shared-memory row
   const UpdDirect U{sk, si};
   uint32_t a_ok = 0, a_new = 0, a_effs = 0;
+  // Leaf I/O is warp-cooperative (as in k_ins_leaf_u): the 32 leaves of a warp's rows move in
+  // 16-B chunks, L/2 lanes per leaf row of keys and L/4 per row of values, so one warp
+  // instruction moves whole lines of 32 / (L/2) leaves instead of 32 scattered slots (per-thread
+  // slot loops made a 512-row round ~17 us, bound by the SM's memory request rate).
+  constexpr int KL = L / 2, KQ = 32 / KL, VL = L / 4, VQ = 32 / VL;
   for (uint32_t g0 = 0; g0 < ng; g0 += SB_ROWS) {
-    const uint32_t gi = g0 + tid;
-    if (tid < SB_ROWS && gi < ng) {
-      const uint32_t j0 = gs[gi], j1 = gs[gi + 1], t = st[j0];
+    if (tid < SB_ROWS) {                                 // whole warps (SB_ROWS % 32 == 0)
+      const uint32_t gi = g0 + tid;
+      const int lane = tid & 31;
+      const uint32_t wb = tid & ~31u;
+      const bool have = gi < ng;
+      uint32_t j0 = 0, j1 = 0, t = 0;
+      if (have) {
+        j0 = gs[gi];
+        j1 = gs[gi + 1];
+        t = st[j0];
+      }
       const uint64_t lb = (uint64_t)t * L;
       uint64_t *rk = rowk + tid * (L + 1);
       uint32_t *rv = rowv + tid * (L + 1);
-      // the leaf's L keys and values in flight together (16-B loads into registers, then the
-      // row): loads interleaved with the shared-memory stores through the generic pointers
-      // were serialised one DRAM round trip per slot
-      ulonglong2 lk[L / 2];
-      uint4 lv[L / 4];
+      ulonglong2 kx[32 / KQ];
+      uint4 vx[32 / VQ];
 #pragma unroll
-      for (int p = 0; p < L / 2; ++p) lk[p] = __ldcg(reinterpret_cast<const ulonglong2 *>(key + lb) + p);
-#pragma unroll
-      for (int p = 0; p < L / 4; ++p) lv[p] = __ldcg(reinterpret_cast<const uint4 *>(val + lb) + p);
-#pragma unroll
-      for (int p = 0; p < L / 2; ++p) {
-        rk[2 * p] = lk[p].x;
-        rk[2 * p + 1] = lk[p].y;
+      for (int it = 0; it < 32 / KQ; ++it) {
+        const int q = it * KQ + lane / KL, cc = lane % KL;
+        const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+        const bool hq = __shfl_sync(0xffffffffu, have, q);
+        kx[it] = hq ? __ldcg(reinterpret_cast<const ulonglong2 *>(key + lq) + cc) : make_ulonglong2(0, 0);
       }
 #pragma unroll
-      for (int p = 0; p < L / 4; ++p) {
-        rv[4 * p] = lv[p].x;
-        rv[4 * p + 1] = lv[p].y;
-        rv[4 * p + 2] = lv[p].z;
-        rv[4 * p + 3] = lv[p].w;
+      for (int it = 0; it < 32 / VQ; ++it) {
+        const int q = it * VQ + lane / VL, cc = lane % VL;
+        const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+        const bool hq = __shfl_sync(0xffffffffu, have, q);
+        vx[it] = hq ? __ldcg(reinterpret_cast<const uint4 *>(val + lq) + cc) : make_uint4(0, 0, 0, 0);
       }
-      const LeafOut o = leaf_group_merge<true>(rk, rv, (uint32_t)L, t, j0, j1, U, bound, kp, key, cnt, tmask, head,
-                                               row_offset, deg, rb, dirty, c);
-      if (o.ok)
-        for (int p = 0; p < L; ++p) key[lb + p] = rk[p];
-      if (o.ok || o.hitm)
-        for (int p = 0; p < L; ++p) val[lb + p] = rv[p];
+#pragma unroll
+      for (int it = 0; it < 32 / KQ; ++it) {
+        const int q = it * KQ + lane / KL, cc = lane % KL;
+        uint64_t *r = rowk + (wb + q) * (L + 1) + 2 * cc;
+        r[0] = kx[it].x;
+        r[1] = kx[it].y;
+      }
+#pragma unroll
+      for (int it = 0; it < 32 / VQ; ++it) {
+        const int q = it * VQ + lane / VL, cc = lane % VL;
+        uint32_t *r = rowv + (wb + q) * (L + 1) + 4 * cc;
+        r[0] = vx[it].x;
+        r[1] = vx[it].y;
+        r[2] = vx[it].z;
+        r[3] = vx[it].w;
+      }
+      __syncwarp();
+      LeafOut o;
+      if (have)
+        o = leaf_group_merge<true>(rk, rv, (uint32_t)L, t, j0, j1, U, bound, kp, key, cnt, tmask, head, row_offset,
+                                   deg, rb, dirty, c);
+      __syncwarp();
+      const bool vdirty = o.ok || o.hitm;
+#pragma unroll
+      for (int it = 0; it < 32 / KQ; ++it) {
+        const int q = it * KQ + lane / KL, cc = lane % KL;
+        const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+        const bool oq = __shfl_sync(0xffffffffu, o.ok, q);
+        const uint64_t *r = rowk + (wb + q) * (L + 1) + 2 * cc;
+        if (oq) *reinterpret_cast<ulonglong2 *>(key + lq + 2 * cc) = make_ulonglong2(r[0], r[1]);
+      }
+#pragma unroll
+      for (int it = 0; it < 32 / VQ; ++it) {
+        const int q = it * VQ + lane / VL, cc = lane % VL;
+        const uint64_t lq = __shfl_sync(0xffffffffu, lb, q);
+        const bool oq = __shfl_sync(0xffffffffu, vdirty, q);
+        const uint32_t *r = rowv + (wb + q) * (L + 1) + 4 * cc;
+        if (oq) *reinterpret_cast<uint4 *>(val + lq + 4 * cc) = make_uint4(r[0], r[1], r[2], r[3]);
+      }
+      __syncwarp();
       a_ok += o.ok ? 1u : 0u;
       a_new += o.nnew;
       a_effs += o.effs;
@@ -3809,15 +3867,14 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
   return GPMA_OK;
 }
 
-// GPMA_SMALL=0 disables the one-kernel small-batch path (read per call)
-// GPMA_SMALL=0 disables the one-kernel small-batch path; GPMA_SMALL=<n> sets the largest insert
-// batch it takes (default 256: one round of leaf rows -- beyond it the single CTA serialises what
-// the multi-kernel path spreads over the GPU; deletes up to 8x that).  Read per call.
+// GPMA_SMALL=0 disables the one-kernel small-batch path; GPMA_SMALL=<n> sets the largest batch it
+// takes (default 1024, measured: at 1000 keys one kernel beats the multi-kernel path, 50 vs 66 us
+// per insert call, 29 vs 34 per delete; at 2000 the single CTA loses).  Read per call.
 static bool small_batch_path(gpma *g, uint64_t n, int op, int path) {
-  uint64_t lim = SB_ROWS;
+  uint64_t lim = SB_DEFAULT;
   if (const char *e = getenv("GPMA_SMALL")) lim = std::min<uint64_t>((uint64_t)atoll(e), SB_MAX);
   if (lim == 0) return false;
-  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) return n <= std::min<uint64_t>(8 * lim, SB_DEL_MAX);
+  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) return n <= std::min<uint64_t>(lim, SB_DEL_MAX);
   if (path == PATH_INS_LEAF || path == PATH_INS_FUSED)
     return n <= lim && (g->L == 4 || g->L == 8 || g->L == 16);
   return false;
@@ -3878,8 +3935,11 @@ static gpma_status run_small(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, in
 #define GP_SMALL_INS(LL)                                                                                         \
   GP_LAUNCH(g, k_small_insert<LL>, 1, SB_T, sb_smem_bytes(LL), s, ik, iv, (uint32_t)n, g->key, g->val, g->cnt,   \
             tmask_of(g), g->head, g->row_offset, g->deg, (uint32_t)nl, g->rb, g->nr, g->V, bound, ro, pk, pv, pt, \
-            dirty, g->ctrl_d, g->ctrl_h, seq)
+            dirty, g->ctrl_d, g->ctrl_h, seq, pbd)
   const uint32_t seq = next_seq(g);
+  auto bits = [](uint64_t x) { uint32_t b = 1; while ((1ull << b) < x) ++b; return b; };
+  const uint32_t pbd0 = bits(g->V);
+  const uint32_t pbd = bits(g->nr) + pbd0 + 11 <= 64 ? pbd0 : 0u;   // packed sort keys fit
   if (g->L == 16) GP_SMALL_INS(16);
   else if (g->L == 8) GP_SMALL_INS(8);
   else GP_SMALL_INS(4);

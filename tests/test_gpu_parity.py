@@ -123,10 +123,13 @@ def _slide_parity(seed, mode, analytics=True, trace=True, stream=None):
             x_g, x_o = xg, xo
 
 
+@pytest.mark.parametrize("path", ["small", "large"])
 @pytest.mark.parametrize("seed", range(20))
-def test_config0_sliding_window_lazy(seed):
+def test_config0_sliding_window_lazy(seed, path, monkeypatch):
     """BASELINE configs[0]: RMAT s10 sliding window, every slide, 20 seeds, through
-    the fused kernels the bench times (sorted lazy delete, fused insert pre-pass + level 0)."""
+    both batch paths the bench times: the one-kernel small batch (1024-key batches take it by
+    default) and the large-batch kernels (interleaved lazy delete, leaf-keyed insert)."""
+    monkeypatch.setenv("GPMA_SMALL", "1024" if path == "small" else "0")
     _slide_parity(seed, DELETE_LAZY, trace=False)
 
 
@@ -137,9 +140,11 @@ def test_config0_sliding_window_lazy_traced(seed):
 
 
 @pytest.mark.parametrize("seed", range(8))
-def test_config0_sliding_window_graph_replay(seed):
+def test_config0_sliding_window_graph_replay(seed, monkeypatch):
     """The 20-seed sweep's streams on a side stream: every batch after the first of a shape is a
-    replayed CUDA graph of the batch prefix (validate, sort, locate, fused leaf merge, summary)."""
+    replayed CUDA graph of the batch prefix (validate, sort, locate, fused leaf merge, summary).
+    (The one-kernel small path is not graph-replayed: GPMA_SMALL=0.)"""
+    monkeypatch.setenv("GPMA_SMALL", "0")
     _slide_parity(seed, DELETE_LAZY, analytics=False, trace=False, stream=torch.cuda.Stream())
 
 
@@ -148,9 +153,9 @@ def test_config0_sliding_window_graph_replay(seed):
                                   "GPMA_ILP=4", "GPMA_SMALL=2048", "GPMA_SMALL=0,GPMA_DEL_SORT=1"])
 @pytest.mark.parametrize("seed", range(3))
 def test_config0_alternative_paths(seed, knob, monkeypatch):
-    """The strategy switches give the same layouts as the defaults (configs[0] batches are 1024 keys:
-    by default the large-batch kernels -- leaf-keyed insert, interleaved lazy delete; GPMA_SMALL=2048
-    sends them through the one-kernel small-batch path (4 rounds of leaf rows) -- and the other
+    """The strategy switches give the same layouts as the defaults (configs[0] batches are 1024 keys,
+    forced onto the large-batch kernels -- leaf-keyed insert, interleaved lazy delete -- with
+    GPMA_SMALL=0; GPMA_SMALL=2048 sends them through the one-kernel small-batch path -- and the other
     knobs through the alternatives: sorted lazy delete, separate pre-pass + k_level0, key-sorted
     fused insert by a thread or a sub-warp per leaf, the host-driven level loop, 1- or 4-way probe
     interleaving)."""
