@@ -1363,6 +1363,27 @@ __global__ void k_pend_gather(const uint32_t *__restrict__ keep, const uint32_t 
   }
 }
 
+// Pending list in key order without a radix sort: the gather left it in leaf order (leaves
+// partition the key space), so only each leaf's own rejected keys -- one group, <= IL_BIG of them,
+// distinct (R10 kept the last copy) -- need ordering.  Thread per entry: its rank among the
+// entries of its leaf.  Writes the level-1 buffers (pk0, pv0, pt0).
+__global__ void k_pend_segsort(const uint64_t *__restrict__ pk1, const uint32_t *__restrict__ pv1,
+                               const uint32_t *__restrict__ pt1, uint64_t p, uint64_t *__restrict__ pk0,
+                               uint32_t *__restrict__ pv0, uint32_t *__restrict__ pt0) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < p; i += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t t = pt1[i];
+    const uint64_t k = pk1[i];
+    uint64_t a = i, b = i + 1;
+    while (a > 0 && pt1[a - 1] == t) --a;
+    while (b < p && pt1[b] == t) ++b;
+    uint64_t r = a;
+    for (uint64_t j = a; j < b; ++j) r += pk1[j] < k ? 1u : 0u;
+    pk0[r] = k;
+    pv0[r] = pv1[i];
+    pt0[r] = t;
+  }
+}
+
 // pending list in key order: values and targets follow the sort's permutation
 __global__ void k_pend_permute(const uint32_t *__restrict__ perm, uint64_t p, const uint32_t *__restrict__ pv_in,
                                const uint32_t *__restrict__ pt_in, uint32_t *__restrict__ pv, uint32_t *__restrict__ pt) {
@@ -3443,7 +3464,14 @@ static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, ui
   a.ctot = (uint64_t *)((char *)g->b_misc2.p + ((sizeof(CoopState) + 63) & ~(size_t)63));
   a.c = g->ctrl_d;
   GP_LAUNCH(g, k_coop_init, 1, 1, 0, s, a.st, p, (uint32_t)cur, lvl, g->ctrl_d, *dirty_base);
-  const int grid = std::max(1, std::min(blocks_per_sm * num_sms(), 4 * num_sms()));
+  // CTAs per SM (GPMA_COOP_CTAS, default 2): every level costs ~8 grid barriers, whose arrival
+  // count serialises on one word; measured 1 / 2 / 4 per SM: configs[2] insert 0.560 / 0.569 /
+  // 0.569 ms, configs[3] grow insert 1.56 / 1.31 / 1.33 ms
+  static const int per_sm = [] {
+    const char *e = getenv("GPMA_COOP_CTAS");
+    return e ? std::max(1, atoi(e)) : 2;
+  }();
+  const int grid = std::max(1, std::min(blocks_per_sm, per_sm) * num_sms());
   void *args[] = {&a};
   g->launches++;
   GP_CHECK(g, cudaLaunchCooperativeKernel((void *)k_levels_coop, grid, CL_T, args, smem, s));
@@ -4211,7 +4239,11 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     g->last.last_slots_rewritten += g->ctrl_h->windows_rewritten * g->L;
     g->last.last_windows_rewritten += g->ctrl_h->windows_rewritten;
     g->last.last_level0_windows = g->ctrl_h->windows_rewritten;
-    if (p_new) {
+    if (p_new && !g->ctrl_h->big) {                    // leaf order: sort inside each leaf only
+      GP_LAUNCH(g, k_pend_segsort, grid_for(p_new), TB, 0, s, pk1, pv1, pt1, p_new, (uint64_t *)g->b_pk[0].p,
+                (uint32_t *)g->b_pv[0].p, (uint32_t *)g->b_pt[0].p);
+      g->last.last_top_level = 1;
+    } else if (p_new) {                                  // (+ oversized groups' keys appended: full sort)
       int sh[8], which = 0;
       const int ns = key_shifts(g->V, sh);
       GP_CHECK(g, radix_sort_pairs(g, pk1, seq, (uint64_t *)g->b_sk[1].p, (uint32_t *)g->b_sv[1].p, p_new, sh, ns, s,
