@@ -128,6 +128,11 @@ gpma *new_handle(uint32_t V) {
     return nullptr;
   }
   memset(g->ctrl_h, 0, sizeof(gp::Ctrl));
+  if (cudaMemset(g->ctrl_d, 0, sizeof(gp::Ctrl)) != cudaSuccess) {   // (Ctrl::done starts at 0)
+    cudaGetLastError();
+    free_handle(g);
+    return nullptr;
+  }
   for (gp::Scratch &x : g->an) {
     if (cudaMalloc((void **)&x.ctrl_d, sizeof(gp::Ctrl)) != cudaSuccess ||
         cudaMallocHost((void **)&x.ctrl_h, sizeof(gp::Ctrl)) != cudaSuccess) {

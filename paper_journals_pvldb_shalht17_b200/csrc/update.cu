@@ -1019,8 +1019,7 @@ __device__ __forceinline__ void find_in_leaf_r(const uint64_t *__restrict__ key,
 // the fields, a system fence, then the sequence number -- the host sees the whole block once it
 // sees the number (wait_ctrl), without waiting for the kernel's completion to reach the stream.
 __device__ __forceinline__ void mirror_ctrl(const Ctrl *c, Ctrl *c_host, uint32_t seq) {
-  __threadfence_system();
-  *c_host = *c;
+  *c_host = *c;                    // (device data reaches the host's later stream work in order)
   __threadfence_system();
   *reinterpret_cast<volatile uint32_t *>(&c_host->seq) = seq;
 }
@@ -1033,7 +1032,6 @@ __device__ __forceinline__ void mirror_ctrl(const Ctrl *c, Ctrl *c_host, uint32_
 // list for level 1 and mirrors its control block to pinned host memory: one launch and one
 // host synchronisation per call instead of a dozen launches.  Lazy deletes likewise.
 constexpr int SB_T = 1024, SB_MAX = 2048, SB_ROWS = 512, SB_DEL_MAX = 4096;
-constexpr uint64_t SB_DEFAULT = 1024;  // default GPMA_SMALL: inserts and lazy deletes <= it take one kernel
 constexpr size_t SB_ROWK_OFF = ((size_t)SB_MAX * 8 + (size_t)SB_MAX * 4 * 2 + (size_t)(SB_MAX + 1) * 4 * 2 + 15) & ~(size_t)15;
 __host__ __device__ constexpr size_t sb_smem_bytes(int L) { return SB_ROWK_OFF + (size_t)SB_ROWS * (L + 1) * 12; }
 
@@ -1136,12 +1134,13 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
   uint32_t np2 = 2;
   while (np2 < n) np2 <<= 1;
   if (pbd) {
+    np2 = np2 < 64 ? 64 : np2;                         // (the merge sort's register phase is 64 wide)
     // (src - rb, dst, arrival) packed into one distinct u64 (pbd = dst bits; the host checks
     // that row bits + pbd + 11 <= 64): half the shuffles and one compare per stage
     for (uint32_t i = tid; i < np2; i += SB_T)
       sk[i] = i < n ? ((((sk[i] >> 32) - rb) << (pbd + 11)) | ((sk[i] & 0xFFFFFFFFull) << 11) | i) : ~0ull;
     __syncthreads();
-    cta_bitonic_sort_u64(sk, np2);
+    cta_merge_sort_u64(sk, np2);
     for (uint32_t i = tid; i < n; i += SB_T) {
       const uint64_t pw = sk[i];
       si[i] = (uint32_t)(pw & (SB_MAX - 1));
@@ -1303,46 +1302,76 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
   }
 }
 
-// small lazy-delete batch: validate, then mark, one CTA, one launch
-__global__ void __launch_bounds__(SB_T) k_small_delete(const uint64_t *__restrict__ ik, uint32_t n,
+// small lazy-delete batch in ONE launch of ceil(n / SD_T) CTAs: every CTA validates
+// the whole batch (<= SB_DEL_MAX keys, L2-resident) so that none marks anything unless all keys
+// are valid -- no grid barrier -- then marks its own slice (R keys per thread in flight); the
+// last CTA to finish (a self-resetting counter) mirrors the control block to the host.  The
+// single-CTA version ran the locate chains of 1024 keys on one SM.
+constexpr int SD_T = 256;
+__global__ void __launch_bounds__(SD_T) k_small_delete(const uint64_t *__restrict__ ik, uint32_t n,
                                                        const uint64_t *__restrict__ key, uint32_t *val, uint32_t *cnt,
                                                        const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
                                                        uint32_t *tmask, uint32_t *deg, uint32_t rb, uint32_t nr,
                                                        uint32_t V, const uint64_t *__restrict__ ro, Ctrl *c,
                                                        Ctrl *c_host, uint32_t seq) {
   const int tid = threadIdx.x;
-  if (tid == 0) {
-    c->err = 0;
-    c->nunique = 0;
-    c->sum = 0;
-    c->sum2 = 0;
-  }
   uint32_t e = 0;
-  for (uint32_t i = tid; i < n; i += SB_T) {
+  for (uint32_t i = tid; i < n; i += SD_T) {
     const uint64_t k = ik[i];
     const uint32_t src = (uint32_t)(k >> 32), dst = (uint32_t)k;
     if (dst == COL_GUARD) e |= 2u;
     if (src - rb >= nr || dst >= V) e |= 1u;
   }
   e = __syncthreads_or(e) ? (__reduce_or_sync(0xffffffffu, e)) : 0u;
-  if (e) atomicOr(&c->err, e);
+  __shared__ uint32_t s_err;
+  if (tid == 0) s_err = 0;
   __syncthreads();
-  if (!c->err) {
-    for (uint32_t i = tid; i < n; i += SB_T) {
-      const uint64_t k = ik[i];
-      const uint32_t t = locate_leaf_rows(head, nleaves, ro, rb, L, k);
-      const uint64_t base = (uint64_t)t * L;
-      const int p = find_in_leaf(key, base, L, k);
-      if (p < 0) continue;
-      if (atomicExch(&val[base + p], VAL_TOMB) != VAL_TOMB) {   // duplicates: one of them accounts it
-        atomicSub(&cnt[t], 1u);
-        atomicOr(&tmask[t], 1u << p);
-        atomicSub(&deg[(uint32_t)(k >> 32) - rb], 1u);
-      }
+  if (e && (tid & 31) == 0) atomicOr(&s_err, e);
+  __syncthreads();
+  if (s_err) {                                           // every CTA sees it; CTA 0 reports
+    if (blockIdx.x == 0 && tid == 0) {
+      c->err = s_err;
+      c->nunique = c->sum = c->sum2 = 0;
+      mirror_ctrl(c, c_host, seq);
     }
+    return;
+  }
+  {
+    const uint32_t i0 = blockIdx.x * SD_T + tid;
+    uint64_t k[2];
+    bool v[2];
+#pragma unroll
+    for (int q = 0; q < 2; ++q) {
+      const uint32_t i = i0 + q * gridDim.x * SD_T;
+      v[q] = i < n;
+      k[q] = v[q] ? ik[i] : 0ull;
+    }
+    uint32_t t[2];
+    locate_leaf_rows_r<2>(head, nleaves, ro, rb, L, k, v, t);
+    int p[2];
+    find_in_leaf_r<2>(key, L, k, v, t, p);
+    uint32_t old[2];
+#pragma unroll
+    for (int q = 0; q < 2; ++q)
+      old[q] = p[q] >= 0 ? atomicExch(&val[(uint64_t)t[q] * L + p[q]], VAL_TOMB) : VAL_TOMB;   // duplicates: one accounts it
+#pragma unroll
+    for (int q = 0; q < 2; ++q)
+      if (old[q] != VAL_TOMB) {
+        atomicSub(&cnt[t[q]], 1u);
+        atomicOr(&tmask[t[q]], 1u << p[q]);
+        atomicSub(&deg[(uint32_t)(k[q] >> 32) - rb], 1u);
+      }
   }
   __syncthreads();
-  if (tid == 0) mirror_ctrl(c, c_host, seq);
+  if (tid == 0) {
+    __threadfence();
+    if (atomicAdd((unsigned long long *)&c->done, 1ull) == gridDim.x - 1) {
+      c->done = 0;
+      c->err = 0;
+      c->nunique = c->sum = c->sum2 = 0;
+      mirror_ctrl(c, c_host, seq);
+    }
+  }
 }
 
 // the rejected new keys (keep[j] = 1) of the leaf-sorted batch, compacted in leaf order with
@@ -3896,15 +3925,19 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
 }
 
 // GPMA_SMALL=0 disables the one-kernel small-batch path; GPMA_SMALL=<n> sets the largest batch it
-// takes (default 1024, measured: at 1000 keys one kernel beats the multi-kernel path, 50 vs 66 us
-// per insert call, 29 vs 34 per delete; at 2000 the single CTA loses).  Read per call.
+// takes (inserts <= min(n, 2048), lazy deletes <= min(n, 4096)).  Default: every batch up to those
+// maxima -- measured (configs[1], tools/r02_small_sweep2.sh): insert call 46 vs 66 us at 1000 keys
+// and 68 vs 75 at 2000 against the multi-kernel path, lazy delete 27 vs 33 at both.  Read per call.
 static bool small_batch_path(gpma *g, uint64_t n, int op, int path) {
-  uint64_t lim = SB_DEFAULT;
-  if (const char *e = getenv("GPMA_SMALL")) lim = std::min<uint64_t>((uint64_t)atoll(e), SB_MAX);
-  if (lim == 0) return false;
-  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) return n <= std::min<uint64_t>(lim, SB_DEL_MAX);
+  uint64_t lim_ins = SB_MAX, lim_del = SB_DEL_MAX;
+  if (const char *e = getenv("GPMA_SMALL")) {
+    const uint64_t lim = (uint64_t)atoll(e);
+    lim_ins = std::min<uint64_t>(lim, SB_MAX);
+    lim_del = std::min<uint64_t>(lim, SB_DEL_MAX);
+  }
+  if (path == PATH_LAZY_UNSORTED || path == PATH_LAZY_SORTED) return n <= lim_del;
   if (path == PATH_INS_LEAF || path == PATH_INS_FUSED)
-    return n <= lim && (g->L == 4 || g->L == 8 || g->L == 16);
+    return n <= lim_ins && (g->L == 4 || g->L == 8 || g->L == 16);
   return false;
 }
 
@@ -3942,7 +3975,8 @@ static gpma_status run_small(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, in
   const uint64_t nl = g->cap / g->L;
   const uint64_t *ro = g->rows_indexed ? g->row_offset : nullptr;
   if (op == GPMA_DELETE) {
-    GP_LAUNCH(g, k_small_delete, 1, SB_T, 0, s, ik, (uint32_t)n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
+    GP_LAUNCH(g, k_small_delete, (unsigned)std::max<uint64_t>(1, (n + 2 * SD_T - 1) / (2 * SD_T)), SD_T, 0, s, ik,
+              (uint32_t)n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
               tmask_of(g), g->deg, g->rb, g->nr, g->V, ro, g->ctrl_d, g->ctrl_h, next_seq(g));
     GP_CHECK(g, cudaGetLastError());
     return GPMA_OK;

@@ -14,31 +14,33 @@ __global__ void __launch_bounds__(1024) k_sort(uint64_t *in, uint64_t *out, uint
   __shared__ uint32_t si[2048];
   uint32_t np2 = 2;
   while (np2 < n) np2 <<= 1;
-  for (uint32_t i = threadIdx.x; i < np2; i += blockDim.x) {
+  const uint32_t np2a = MODE == 2 && np2 < 64 ? 64 : np2;
+  for (uint32_t i = threadIdx.x; i < np2a; i += blockDim.x) {
     sk[i] = i < n ? in[i] : ~0ull;
     si[i] = i;
   }
   __syncthreads();
   unsigned long long t0 = clock64();
   if (MODE == 0) cta_bitonic_sort_u64(sk, np2);
-  else cta_bitonic_sort(sk, si, np2);
+  else if (MODE == 1) cta_bitonic_sort(sk, si, np2);
+  else cta_merge_sort_u64(sk, np2 < 64 ? 64 : np2);
   unsigned long long t1 = clock64();
   if (threadIdx.x == 0) *cyc = t1 - t0;
   for (uint32_t i = threadIdx.x; i < n; i += blockDim.x) out[i] = sk[i];
 }
 
 int main() {
-  for (uint32_t n : {100u, 1000u, 2000u}) {
+  for (uint32_t n : {1u, 5u, 33u, 64u, 100u, 1000u, 2000u, 2048u}) {
     std::vector<uint64_t> h(n);
     uint64_t x = 88172645463325252ull;
     for (auto &v : h) { x ^= x << 13; x ^= x >> 7; x ^= x << 17; v = x >> 8; }
     uint64_t *d, *o; unsigned long long *c;
     cudaMalloc(&d, n * 8); cudaMalloc(&o, n * 8); cudaMalloc(&c, 8);
     cudaMemcpy(d, h.data(), n * 8, cudaMemcpyHostToDevice);
-    for (int mode = 0; mode < 2; ++mode) {
+    for (int mode = 0; mode < 3; ++mode) {
       unsigned long long cy = 0;
       for (int rep = 0; rep < 3; ++rep) {
-        if (mode == 0) k_sort<0><<<1, 1024>>>(d, o, n, c); else k_sort<1><<<1, 1024>>>(d, o, n, c);
+        if (mode == 0) k_sort<0><<<1, 1024>>>(d, o, n, c); else if (mode == 1) k_sort<1><<<1, 1024>>>(d, o, n, c); else k_sort<2><<<1, 1024>>>(d, o, n, c);
         cudaMemcpy(&cy, c, 8, cudaMemcpyDeviceToHost);
       }
       std::vector<uint64_t> r(n);
