@@ -146,6 +146,47 @@ def test_small_path_sizes_and_stability(n, monkeypatch):
     assert_same_csr(g, o)
 
 
+@pytest.mark.parametrize("bad_at", [0, 1500, 2999])
+def test_multi_cta_small_delete_rejects_whole_batch(bad_at):
+    """A 3000-key lazy delete takes the multi-CTA one-kernel path (6 CTAs): one invalid key
+    anywhere -- in another CTA's slice -- must leave the store untouched (every CTA validates
+    the whole batch before any marks), and the valid batch then deletes exactly the live keys."""
+    from paper_journals_pvldb_shalht17_b200 import GpmaError
+    rng = np.random.default_rng(5 + bad_at)
+    V = 1 << 11
+    k0 = np.unique(rng.integers(0, V, 20000) << 32 | rng.integers(0, V, 20000)).astype(np.uint64).tolist()
+    g, o = _pair(V, k0, [1] * len(k0))
+    dk = [k0[i] for i in rng.integers(0, len(k0), 3000)]
+    bad = list(dk)
+    bad[bad_at] = (V + 3) << 32 | 1                    # src out of range
+    with pytest.raises(GpmaError):
+        g.delete(keys_t(bad))
+    assert_same_layout(g, o)
+    _apply(g, o, dk, op=1)
+    assert_same_csr(g, o)
+
+
+@pytest.mark.parametrize("direct", ["1", "0"])
+def test_large_device_batch_direct_vs_staged(direct, monkeypatch):
+    """Batches of >= 2^16 device keys on the read-only paths (leaf-keyed insert, unsorted lazy
+    delete) can be read in place without staging or graph replay (GPMA_DIRECT=1); the default
+    staged / graph-replayed path (0) must give the same layouts, with duplicates (R10) and
+    deletes of absent keys."""
+    monkeypatch.setenv("GPMA_DIRECT", direct)
+    rng = np.random.default_rng(404)
+    V = 1 << 13
+    k0 = np.unique(rng.integers(0, V, 150000) << 32 | rng.integers(0, V, 150000)).astype(np.uint64).tolist()
+    g, o = _pair(V, k0, [1] * len(k0))
+    for step in range(3):
+        n = 70000 + 1000 * step
+        ks = (rng.integers(0, V, n) << 32 | rng.integers(0, V, n)).astype(np.uint64).tolist()
+        vs = rng.integers(0, 1 << 31, n).tolist()
+        _apply(g, o, ks, vs)
+        dk = [k0[i] for i in rng.integers(0, len(k0), n)]
+        _apply(g, o, dk, op=1)
+    assert_same_csr(g, o)
+
+
 def test_torch_allocator_hooks():
     """gpma_config.alloc/free through PyTorch's caching allocator (SURVEY §8(b) "Ownership"): the
     store lives in torch's pool while the handle lives, the results are unchanged, and destroy
