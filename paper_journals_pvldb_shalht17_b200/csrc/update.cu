@@ -934,7 +934,8 @@ __global__ void __launch_bounds__(ILU_T) k_ins_leaf_u(const uint64_t *__restrict
 template <int R>
 __device__ __forceinline__ void locate_leaf_rows_r(const uint64_t *__restrict__ head, uint32_t nleaves,
                                                    const uint64_t *__restrict__ ro, uint32_t rb, uint32_t L,
-                                                   const uint64_t (&k)[R], const bool (&v)[R], uint32_t (&t)[R]) {
+                                                   const uint64_t (&k)[R], const bool (&v)[R], uint32_t (&t)[R],
+                                                   float fv = 0.f) {
   uint32_t lo[R], hi[R], a[R];
   if (!ro) {
 #pragma unroll
@@ -954,6 +955,45 @@ __device__ __forceinline__ void locate_leaf_rows_r(const uint64_t *__restrict__ 
     a[q] = (uint32_t)leaf_div(r[q].x, L);
     lo[q] = a[q] + 1;
     hi[q] = v[q] ? min((uint32_t)leaf_div(r[q].y, L) + 1, nleaves) : a[q];
+  }
+  if (fv > 0.f) {
+    // Interpolation step for rows over more than 8 leaves (fv = 1/V): the row's keys are sorted
+    // by dst, so the leaf of (u, dst) sits near a + dst/V * (row leaves).  The aligned 64-B line
+    // of 8 heads around that guess is read in one access; it either brackets the answer (done)
+    // or cuts the range at its edge.  Replaces the ~5 dependent head probes an RMAT delete made
+    // (edge-weighted row spans are hundreds of leaves) by about one; exact for any data (a bad
+    // guess only leaves more range for the binary search below).
+    ulonglong2 hl[R][4];
+    uint32_t ls[R];
+    bool use[R];
+#pragma unroll
+    for (int q = 0; q < R; ++q) {
+      use[q] = v[q] && hi[q] > lo[q] + 8;
+      uint32_t g = a[q] + (uint32_t)((float)(uint32_t)k[q] * fv * (float)(hi[q] - a[q]));
+      g = min(max(g, lo[q]), hi[q] - 1);
+      ls[q] = g & ~7u;
+#pragma unroll
+      for (int j = 0; j < 4; ++j)
+        hl[q][j] = use[q] ? __ldg(reinterpret_cast<const ulonglong2 *>(head + ls[q]) + j) : make_ulonglong2(0, 0);
+    }
+#pragma unroll
+    for (int q = 0; q < R; ++q) {
+      if (!use[q]) continue;
+      const uint32_t wlo = max(ls[q], lo[q]), whi = min(ls[q] + 8, hi[q]);
+      uint32_t cnt = 0;
+#pragma unroll
+      for (int j = 0; j < 8; ++j) {
+        const uint32_t idx = ls[q] + j;
+        const uint64_t h = (j & 1) ? hl[q][j >> 1].y : hl[q][j >> 1].x;
+        cnt += (idx >= wlo && idx < whi && h <= k[q]) ? 1u : 0u;
+      }
+      if (cnt < whi - wlo) {                             // a head > k inside the line
+        if (cnt > 0 || wlo == lo[q]) lo[q] = hi[q] = wlo + cnt;
+        else hi[q] = wlo;
+      } else {
+        lo[q] = whi;
+      }
+    }
   }
   bool any = true;
   while (any) {
@@ -1070,7 +1110,7 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
                                                        uint32_t *deg, uint32_t nleaves, uint32_t rb, uint32_t nr,
                                                        uint32_t V, uint32_t bound, const uint64_t *__restrict__ ro,
                                                        uint64_t *pk, uint32_t *pv, uint32_t *pt, uint2 *dirty, Ctrl *c,
-                                                       Ctrl *c_host, uint32_t seq, uint32_t pbd) {
+                                                       Ctrl *c_host, uint32_t seq, uint32_t pbd, float fv) {
   extern __shared__ __align__(16) unsigned char sb_smem[];
   uint64_t *sk = reinterpret_cast<uint64_t *>(sb_smem);           // [SB_MAX] keys (sorted)
   uint32_t *si = reinterpret_cast<uint32_t *>(sk + SB_MAX);       // [SB_MAX] arrival index -> sorted values
@@ -1117,7 +1157,7 @@ __global__ void __launch_bounds__(SB_T) k_small_insert(const uint64_t *__restric
       }
     }
     uint32_t t[2];
-    locate_leaf_rows_r<2>(head, nleaves, ro, rb, L, k, v, t);
+    locate_leaf_rows_r<2>(head, nleaves, ro, rb, L, k, v, t, fv);
     for (int q = 0; q < 2; ++q) {
       const uint32_t i = tid + q * SB_T;
       if (i < n) gs[i] = t[q];
@@ -1313,7 +1353,7 @@ __global__ void __launch_bounds__(SD_T) k_small_delete(const uint64_t *__restric
                                                        const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
                                                        uint32_t *tmask, uint32_t *deg, uint32_t rb, uint32_t nr,
                                                        uint32_t V, const uint64_t *__restrict__ ro, Ctrl *c,
-                                                       Ctrl *c_host, uint32_t seq) {
+                                                       Ctrl *c_host, uint32_t seq, float fv) {
   const int tid = threadIdx.x;
   uint32_t e = 0;
   for (uint32_t i = tid; i < n; i += SD_T) {
@@ -1347,7 +1387,7 @@ __global__ void __launch_bounds__(SD_T) k_small_delete(const uint64_t *__restric
       k[q] = v[q] ? ik[i] : 0ull;
     }
     uint32_t t[2];
-    locate_leaf_rows_r<2>(head, nleaves, ro, rb, L, k, v, t);
+    locate_leaf_rows_r<2>(head, nleaves, ro, rb, L, k, v, t, fv);
     int p[2];
     find_in_leaf_r<2>(key, L, k, v, t, p);
     uint32_t old[2];
@@ -1432,7 +1472,7 @@ __global__ void __launch_bounds__(256) k_lazy_delete_r(const uint64_t *__restric
                                                        uint32_t *__restrict__ cnt, const uint64_t *__restrict__ head,
                                                        uint32_t nleaves, uint32_t L, uint32_t *__restrict__ tmask,
                                                        uint32_t *__restrict__ deg, uint32_t rb, const Ctrl *c,
-                                                       const uint64_t *__restrict__ ro) {
+                                                       const uint64_t *__restrict__ ro, float fv) {
   if (c->err) return;
   const uint64_t nthr = (uint64_t)gridDim.x * blockDim.x;
   for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i0 < n; i0 += nthr * LD_R) {
@@ -1445,7 +1485,7 @@ __global__ void __launch_bounds__(256) k_lazy_delete_r(const uint64_t *__restric
       k[q] = v[q] ? keys[i] : 0ull;
     }
     uint32_t t[LD_R];
-    locate_leaf_rows_r<LD_R>(head, nleaves, ro, rb, L, k, v, t);
+    locate_leaf_rows_r<LD_R>(head, nleaves, ro, rb, L, k, v, t, fv);
     int p[LD_R];
     find_in_leaf_r<LD_R>(key, L, k, v, t, p);
     // one exchange per found key: the copy that swaps a live value for TOMB accounts it
@@ -1470,7 +1510,7 @@ __global__ void __launch_bounds__(256) k_locate_u_r(const uint64_t *__restrict__
                                                     const uint64_t *__restrict__ head, uint32_t nleaves, uint32_t L,
                                                     uint32_t rb, const uint64_t *__restrict__ ro,
                                                     uint64_t *__restrict__ tk, uint32_t *__restrict__ tix,
-                                                    const Ctrl *c) {
+                                                    const Ctrl *c, float fv) {
   if (c->err) return;
   const uint64_t nthr = (uint64_t)gridDim.x * blockDim.x;
   for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i0 < n; i0 += nthr * LD_R) {
@@ -1483,7 +1523,7 @@ __global__ void __launch_bounds__(256) k_locate_u_r(const uint64_t *__restrict__
       k[q] = v[q] ? ik[i] : 0ull;
     }
     uint32_t t[LD_R];
-    locate_leaf_rows_r<LD_R>(head, nleaves, ro, rb, L, k, v, t);
+    locate_leaf_rows_r<LD_R>(head, nleaves, ro, rb, L, k, v, t, fv);
 #pragma unroll
     for (int q = 0; q < LD_R; ++q) {
       const uint64_t i = i0 + (uint64_t)q * nthr;
@@ -3008,7 +3048,7 @@ static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v
   cudaError_t e1 = dev_alloc(g, (void **)k, cap * 8, s);
   cudaError_t e2 = dev_alloc(g, (void **)v, cap * 4, s);
   cudaError_t e3 = dev_alloc(g, (void **)c, nl * 12, s);  // live counts, tombstone masks, guards
-  cudaError_t e4 = dev_alloc(g, (void **)hd, nl * 8, s);
+  cudaError_t e4 = dev_alloc(g, (void **)hd, ((nl + 7) & ~(uint64_t)7) * 8, s);   // (whole 64-B lines)
   if ((e1 || e2 || e3 || e4) && g->spare.key) {          // out of memory: give the spare set back first
     dev_free(g, *k, s);
     dev_free(g, *v, s);
@@ -3018,7 +3058,7 @@ static gpma_status alloc_store(gpma *g, uint64_t cap, uint64_t **k, uint32_t **v
     e1 = dev_alloc(g, (void **)k, cap * 8, s);
     e2 = dev_alloc(g, (void **)v, cap * 4, s);
     e3 = dev_alloc(g, (void **)c, nl * 12, s);
-    e4 = dev_alloc(g, (void **)hd, nl * 8, s);
+    e4 = dev_alloc(g, (void **)hd, ((nl + 7) & ~(uint64_t)7) * 8, s);
   }
   if (e1 || e2 || e3 || e4) {
     cudaGetLastError();
@@ -3787,6 +3827,14 @@ static int leaf_shifts(uint64_t nleaves, int *sh) {
 //  * otherwise (strict deletes, GPMA lock-based inserts, traced batches): sort -> pre-pass ->
 //    compact -> level 0 (k_level0) unless traced -> summary.
 // *srt = the sorted batch.
+// 1/V for the interpolation step of the row search (GPMA_INTERP=0: plain binary search; read per
+// call).  Every located key has dst < V.
+static float interp_fv(gpma *g) {
+  const char *e = getenv("GPMA_INTERP");
+  if (e && atoi(e) == 0) return 0.f;
+  return 1.0f / (float)std::max<uint32_t>(g->V, 1u);
+}
+
 static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, int op, Sorted *srt,
                               cudaStream_t s) {
   gpma_status st;
@@ -3800,10 +3848,10 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
     const int R = ilp_r();
     if (R >= 4)
       GP_LAUNCH(g, k_lazy_delete_r<4>, grid_for((n + 3) / 4), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head,
-                (uint32_t)nl, g->L, tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
+                (uint32_t)nl, g->L, tmask_of(g), g->deg, g->rb, g->ctrl_d, ro, interp_fv(g));
     else if (R == 2)
       GP_LAUNCH(g, k_lazy_delete_r<2>, grid_for((n + 1) / 2), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head,
-                (uint32_t)nl, g->L, tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
+                (uint32_t)nl, g->L, tmask_of(g), g->deg, g->rb, g->ctrl_d, ro, interp_fv(g));
     else
       GP_LAUNCH(g, k_lazy_delete, grid_for(n), TB, 0, s, ik, n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
                 tmask_of(g), g->deg, g->rb, g->ctrl_d, ro);
@@ -3825,10 +3873,10 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
     const int R = ilp_r();
     if (R >= 4)
       GP_LAUNCH(g, k_locate_u_r<4>, grid_for((n + 3) / 4), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0,
-                tx0, g->ctrl_d);
+                tx0, g->ctrl_d, interp_fv(g));
     else if (R == 2)
       GP_LAUNCH(g, k_locate_u_r<2>, grid_for((n + 1) / 2), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0,
-                tx0, g->ctrl_d);
+                tx0, g->ctrl_d, interp_fv(g));
     else
       GP_LAUNCH(g, k_locate_u, grid_for(n), TB, 0, s, ik, n, g->head, (uint32_t)nl, g->L, g->rb, ro, tk0, tx0, g->ctrl_d);
     int sh[8], which = 0;
@@ -3977,7 +4025,7 @@ static gpma_status run_small(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, in
   if (op == GPMA_DELETE) {
     GP_LAUNCH(g, k_small_delete, (unsigned)std::max<uint64_t>(1, (n + 2 * SD_T - 1) / (2 * SD_T)), SD_T, 0, s, ik,
               (uint32_t)n, g->key, g->val, g->cnt, g->head, (uint32_t)nl, g->L,
-              tmask_of(g), g->deg, g->rb, g->nr, g->V, ro, g->ctrl_d, g->ctrl_h, next_seq(g));
+              tmask_of(g), g->deg, g->rb, g->nr, g->V, ro, g->ctrl_d, g->ctrl_h, next_seq(g), interp_fv(g));
     GP_CHECK(g, cudaGetLastError());
     return GPMA_OK;
   }
@@ -3997,7 +4045,7 @@ static gpma_status run_small(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, in
 #define GP_SMALL_INS(LL)                                                                                         \
   GP_LAUNCH(g, k_small_insert<LL>, 1, SB_T, sb_smem_bytes(LL), s, ik, iv, (uint32_t)n, g->key, g->val, g->cnt,   \
             tmask_of(g), g->head, g->row_offset, g->deg, (uint32_t)nl, g->rb, g->nr, g->V, bound, ro, pk, pv, pt, \
-            dirty, g->ctrl_d, g->ctrl_h, seq, pbd)
+            dirty, g->ctrl_d, g->ctrl_h, seq, pbd, interp_fv(g))
   const uint32_t seq = next_seq(g);
   auto bits = [](uint64_t x) { uint32_t b = 1; while ((1ull << b) < x) ++b; return b; };
   const uint32_t pbd0 = bits(g->V);
