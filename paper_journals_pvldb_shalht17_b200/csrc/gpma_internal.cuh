@@ -354,6 +354,7 @@ struct gpma {
   gp::Ctrl *ctrl_d = nullptr;
   gp::Ctrl *ctrl_h = nullptr;     // pinned mirror
   uint32_t ctrl_seq = 0;          // sequence number of the last mirrored one-kernel call
+  uint64_t root_need = 0;         // entries of a root re-layout (live + pending): its scratch size
   void *pin = nullptr;            // 256 B of pinned host scratch (read-backs of small device state)
   gp::Scratch an[gp::AN_N];       // analytics (read-only on the store)
 

@@ -6,6 +6,8 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <chrono>
+#include <cstdio>
 #include <cstring>
 
 #include "gpma_internal.cuh"
@@ -77,17 +79,40 @@ void pool_detach(gpma *g) {
   g->pool_attached = false;
 }
 
+// GPMA_TRACE_ALLOC=1: every allocation >= 64 MiB with its host time on stderr (diagnostics)
+static bool trace_alloc() {
+  static const bool on = [] {
+    const char *e = getenv("GPMA_TRACE_ALLOC");
+    return e && atoi(e) != 0;
+  }();
+  return on;
+}
+
 cudaError_t dev_alloc(gpma *g, void **p, size_t bytes, cudaStream_t s) {
   *p = nullptr;
+  const auto t0 = std::chrono::steady_clock::now();
+  cudaError_t e;
   if (g->alloc_fn) {
     *p = g->alloc_fn(bytes, (gpma_stream_t)s, g->alloc_ctx);
-    return *p ? cudaSuccess : cudaErrorMemoryAllocation;
+    e = *p ? cudaSuccess : cudaErrorMemoryAllocation;
+  } else {
+    cudaMemPool_t pool = lib_pool(g->device);
+    e = pool ? cudaMallocFromPoolAsync(p, bytes, pool, s) : cudaMallocAsync(p, bytes, s);
+    if (e != cudaSuccess) {
+      cudaGetLastError();
+      *p = nullptr;
+    }
   }
-  cudaMemPool_t pool = lib_pool(g->device);
-  cudaError_t e = pool ? cudaMallocFromPoolAsync(p, bytes, pool, s) : cudaMallocAsync(p, bytes, s);
-  if (e != cudaSuccess) {
-    cudaGetLastError();
-    *p = nullptr;
+  if (trace_alloc() && bytes >= (64u << 20)) {
+    uint64_t res = 0, used = 0;
+    if (!g->alloc_fn) {
+      cudaMemPool_t pool = lib_pool(g->device);
+      cudaMemPoolGetAttribute(pool, cudaMemPoolAttrReservedMemCurrent, &res);
+      cudaMemPoolGetAttribute(pool, cudaMemPoolAttrUsedMemCurrent, &used);
+    }
+    fprintf(stderr, "[gpma] dev_alloc %.1f MiB: %.3f ms (%s; pool reserved %.0f used %.0f MiB)\n", bytes / 1048576.0,
+            std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count(),
+            e == cudaSuccess ? "ok" : "failed", res / 1048576.0, used / 1048576.0);
   }
   return e;
 }
@@ -106,7 +131,16 @@ void dev_free(gpma *g, void *p, cudaStream_t s) {
 cudaError_t ensure(gpma *g, DevBuf &b, size_t bytes, cudaStream_t s) {
   if (bytes == 0) bytes = 16;
   if (b.bytes >= bytes) return cudaSuccess;
-  const size_t want = std::max(bytes, b.bytes + b.bytes / 2);
+  size_t want = std::max(bytes, b.bytes + b.bytes / 2);
+  // Large scratch in power-of-two sizes: the pool serves a request from one free chunk, and
+  // chunks freed by a previous store / scratch of another size made it re-map fragmented free
+  // memory (8-14 ms per 256-512 MiB request with the pool's reserved size unchanged,
+  // tools/resize_trace.py with GPMA_TRACE_ALLOC=1); equal size classes reuse whole chunks.
+  if (want >= (64u << 20)) {
+    size_t p2 = 64u << 20;
+    while (p2 < want) p2 <<= 1;
+    want = p2;
+  }
   dev_free(g, b.p, s);
   b.p = nullptr;
   b.bytes = 0;

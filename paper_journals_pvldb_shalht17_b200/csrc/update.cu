@@ -18,6 +18,8 @@
 #include <cooperative_groups.h>
 
 #include <algorithm>
+#include <chrono>
+#include <cstdio>
 #include <atomic>
 
 #include "gpma_internal.cuh"
@@ -3276,8 +3278,22 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     GP_LAUNCH(g, k_lvl_merge_small, (unsigned)wins_bound, LM_T, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
               g->row_offset, (uint2 *)g->b_dirty.p, *dirty_base);
   } else {
-    // scratch: sum of merged window sizes <= wins_bound * wslots (and <= cap + p)
-    uint64_t need = a.force ? g->cap + p : wins_bound * wslots;
+    // Windows of >= GB_CHUNK slots (the host-driven high levels): read the number of accepted
+    // windows first -- a root-bound batch (every level rejects) then skips the merge kernels,
+    // and the scratch is sized by the accepted windows, not by every window holding pending
+    // updates (which had allocated up to half the store's bytes at level h-1 for nothing).
+    uint64_t nacc_h = wins_bound;
+    if (!a.force && !small && wslots >= (uint64_t)GB_CHUNK) {
+      GP_CHECK(g, readback(g, g->pin, a.aidx + p, 4, s));
+      GP_CHECK(g, cudaStreamSynchronize(s));
+      uint32_t na;
+      memcpy(&na, g->pin, 4);
+      nacc_h = na;
+    }
+    if (nacc_h == 0) goto merged;
+  {
+    // scratch: sum of merged window sizes <= accepted windows * wslots (and <= cap + p)
+    uint64_t need = a.force ? (g->root_need ? g->root_need : g->cap + p) : nacc_h * wslots;
     GP_CHECK(g, ensure(g, g->b_wk, need * 8, s));
     GP_CHECK(g, ensure(g, g->b_wv, need * 4, s));
     a.wk = (uint64_t *)g->b_wk.p;
@@ -3292,7 +3308,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
       GP_LAUNCH(g, k_lvl_leafcnt, grid_for(lb), TB, 0, s, a, g->cnt, lb);
       GP_CHECK(g, scan_u64(g, a.lpre, a.lpre, lb, s));
     }
-    uint64_t bslots = wins_bound * wslots;
+    uint64_t bslots = (a.force ? wins_bound : nacc_h) * wslots;
     uint64_t bslots_r = (bslots + 31) & ~31ull;
     if (a.lvl && wslots >= (uint64_t)GB_CHUNK && gather_big_on()) {
       const uint64_t nch = bslots / GB_CHUNK;
@@ -3316,6 +3332,8 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
                 g->row_offset, g->L, nl_new, g->rb);
     }
   }
+  }
+merged:
   if (small) {
     GP_LAUNCH(g, k_lvl_back_small, 1, LS_T, 0, s, a, g->ctrl_d);
   } else {
@@ -3406,8 +3424,35 @@ static Lvl make_lvl(gpma *g, int cur, uint64_t p, uint32_t lvl, int op) {
 // Root resize (Alg. 4 l.16-17; R14): double until the live entries plus the pending
 // insertions fit max_h of the new capacity; halve (strict deletes) while below min_h
 // and cap > 2L.  Everything is laid out evenly over the new array.
+// GPMA_TRACE_ALLOC=1: phase times of a root resize on stderr (the stream synchronised at each
+// stamp -- diagnostics only)
+static thread_local std::chrono::steady_clock::time_point tl_call_start;
+struct ResizeTrace {
+  bool on;
+  cudaStream_t s;
+  std::chrono::steady_clock::time_point t;
+  explicit ResizeTrace(cudaStream_t s_) : s(s_) {
+    const char *e = getenv("GPMA_TRACE_ALLOC");
+    on = e && atoi(e) != 0;
+    if (on) {
+      cudaStreamSynchronize(s);
+      t = std::chrono::steady_clock::now();
+      fprintf(stderr, "[gpma] resize %-12s %.3f ms\n", "levels<root",
+              std::chrono::duration<double, std::milli>(t - tl_call_start).count());
+    }
+  }
+  void stamp(const char *what) {
+    if (!on) return;
+    cudaStreamSynchronize(s);
+    const auto n = std::chrono::steady_clock::now();
+    fprintf(stderr, "[gpma] resize %-12s %.3f ms\n", what, std::chrono::duration<double, std::milli>(n - t).count());
+    t = n;
+  }
+};
+
 static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, uint64_t *dirty_base) {
   Nvtx nvtx_("update: root resize");
+  ResizeTrace tr(s);
   gpma_status st;
   uint64_t nl = g->cap / g->L;
   if ((st = zero_ctrl(g, s))) return st;
@@ -3437,13 +3482,19 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   uint64_t *nk = g->key;
   uint32_t *nv = g->val, *ncnt = g->cnt;
   uint64_t *nhead = g->head;
+  tr.stamp("count");
   if (cap != g->cap) {
     if ((st = alloc_store(g, cap, &nk, &nv, &ncnt, &nhead, s))) return st;
   }
+  tr.stamp("alloc_store");
   Lvl a = make_lvl(g, cur, p, g->h, op);
   a.force = 1;
   LevelOut lo{};
-  if ((st = level_step(g, a, cur, &lo, dirty_base, s, true, cap, nk, nv, ncnt))) return st;
+  g->root_need = ntot + p;                 // the dense root list: live entries + the pending
+  st = level_step(g, a, cur, &lo, dirty_base, s, true, cap, nk, nv, ncnt);
+  g->root_need = 0;
+  if (st) return st;
+  tr.stamp("root_merge");
   if (cap != g->cap) {
     if (spare_on()) {
       spare_stash(g, g->cap, g->key, g->val, g->cnt, g->head, s);
@@ -3460,10 +3511,13 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
     g->resizes++;
     g->last.last_resized = 1;
   }
+  tr.stamp("free/stash");
   set_geometry(g, cap);
   g->last.last_slots_rewritten += cap;
   g->last.last_windows_rewritten += 1;
-  return recompute_heads(g, s);
+  st = recompute_heads(g, s);
+  tr.stamp("heads");
+  return st;
 }
 
 // ---- the device-resident level loop from the host
@@ -4175,6 +4229,7 @@ gpma_status update_batch(gpma *g, const uint64_t *keys, const uint32_t *vals, ui
   g->last = gpma_stats_t{};
   g->trace.clear();
   if (n == 0) return GPMA_OK;
+  tl_call_start = std::chrono::steady_clock::now();
   int path = prefix_path(g, op);
   Sorted srt;
   Nvtx nvtx_(op == GPMA_INSERT ? "update: insert prefix" : "update: delete prefix");
