@@ -118,6 +118,10 @@ gpma *new_handle(uint32_t V) {
   gpma *g = new (std::nothrow) gpma();
   if (!g) return nullptr;
   g->V = V;
+  if (const char *e = getenv("GPMA_L2_FETCH")) {     // L2 fetch granularity (bytes) of the context
+    cudaDeviceSetLimit(cudaLimitMaxL2FetchGranularity, (size_t)atoi(e));
+    cudaGetLastError();
+  }
   if (cudaMalloc((void **)&g->ctrl_d, sizeof(gp::Ctrl)) != cudaSuccess ||
       cudaMallocHost((void **)&g->ctrl_h, sizeof(gp::Ctrl)) != cudaSuccess ||
       cudaMallocHost(&g->pin, 256) != cudaSuccess) {

@@ -10,6 +10,7 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 #include <stdio.h>
+#include <stdlib.h>
 
 __device__ __forceinline__ uint64_t mix(uint64_t z) {
   z += 0x9E3779B97F4A7C15ull;
@@ -18,7 +19,17 @@ __device__ __forceinline__ uint64_t mix(uint64_t z) {
   return z ^ (z >> 31);
 }
 
-template <int G, int R>
+template <int M>
+__device__ __forceinline__ uint4 ld16(const uint4 *p) {
+  if (M == 0) return __ldg(p);                 // ld.global.nc (read-only / texture path)
+  if (M == 1) return __ldcg(p);                // ld.global.cg (L2 only)
+  if (M == 2) return __ldcs(p);                // ld.global.cs (streaming)
+  uint4 v;                                     // ld.global (weak, L1-cached)
+  asm volatile("ld.global.v4.u32 {%0,%1,%2,%3}, [%4];" : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "l"(p));
+  return v;
+}
+
+template <int G, int R, int M = 0>
 __global__ void __launch_bounds__(256) k_read(const uint4 *__restrict__ a, uint64_t nlines, uint64_t nops,
                                               uint64_t seed, uint4 *sink) {
   constexpr int W = G / 16;
@@ -29,9 +40,9 @@ __global__ void __launch_bounds__(256) k_read(const uint4 *__restrict__ a, uint6
 #pragma unroll
     for (int q = 0; q < R; ++q) {
       const uint64_t i = i0 + q * nthr;
-      const uint64_t line = mix(i ^ seed) % nlines;
+      const uint64_t line = mix(i ^ seed) & (nlines - 1);   // (sizes are powers of two)
 #pragma unroll
-      for (int w = 0; w < W; ++w) v[q][w] = i < nops ? __ldg(a + line * W + w) : make_uint4(0, 0, 0, 0);
+      for (int w = 0; w < W; ++w) v[q][w] = i < nops ? ld16<M>(a + line * W + w) : make_uint4(0, 0, 0, 0);
     }
 #pragma unroll
     for (int q = 0; q < R; ++q)
@@ -48,11 +59,33 @@ __global__ void __launch_bounds__(256) k_atomic(uint32_t *a, uint64_t n, uint64_
   uint32_t acc = 0;
   const uint64_t nthr = (uint64_t)gridDim.x * blockDim.x;
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < nops; i += nthr) {
-    const uint64_t j = mix(i ^ seed) % n;
+    const uint64_t j = mix(i ^ seed) & (n - 1);
     if (RET) acc += atomicAdd(a + j, 1u);
     else atomicAdd(a + j, 1u);
   }
   if (RET && acc == 0x12345678u) sink[0] = acc;
+}
+
+// read-modify-write of a random aligned G-byte line (the leaf rewrite of the insert kernel)
+template <int G, int R>
+__global__ void __launch_bounds__(256) k_line_rmw(uint4 *a, uint64_t nlines, uint64_t nops, uint64_t seed) {
+  constexpr int W = G / 16;
+  const uint64_t nthr = (uint64_t)gridDim.x * blockDim.x;
+  for (uint64_t i0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i0 < nops; i0 += nthr * R) {
+    uint64_t line[R];
+    uint4 v[R][W];
+#pragma unroll
+    for (int q = 0; q < R; ++q) {
+      line[q] = mix((i0 + q * nthr) ^ seed) & (nlines - 1);
+#pragma unroll
+      for (int w = 0; w < W; ++w) v[q][w] = i0 + q * nthr < nops ? a[line[q] * W + w] : make_uint4(0, 0, 0, 0);
+    }
+#pragma unroll
+    for (int q = 0; q < R; ++q)
+      if (i0 + q * nthr < nops)
+#pragma unroll
+        for (int w = 0; w < W; ++w) { v[q][w].x += 1; a[line[q] * W + w] = v[q][w]; }
+  }
 }
 
 __global__ void k_copy(const uint4 *__restrict__ a, uint4 *__restrict__ b, uint64_t n) {
@@ -86,13 +119,13 @@ static float timeit(F f) {
   return best;
 }
 
-template <int G>
+template <int G, int R = 4, int M = 0>
 static void read_case(const uint4 *a, uint64_t bytes, uint64_t nops, uint4 *sink, int blocks) {
   const uint64_t nl = bytes / G;
-  const float ms = timeit([&] { k_read<G, 4><<<blocks, 256>>>(a, nl, nops, 7, sink); });
-  printf("{\"kind\": \"read\", \"granule_B\": %d, \"array_MB\": %llu, \"ops\": %llu, \"ms\": %.4f, \"Gops_s\": %.3f, "
+  const float ms = timeit([&] { k_read<G, R, M><<<blocks, 256>>>(a, nl, nops, 7, sink); });
+  printf("{\"kind\": \"read\", \"ldmode\": %d, \"ilp\": %d, \"granule_B\": %d, \"array_MB\": %llu, \"ops\": %llu, \"ms\": %.4f, \"Gops_s\": %.3f, "
          "\"GB_s_at_granule\": %.1f}\n",
-         G, (unsigned long long)(bytes >> 20), (unsigned long long)nops, ms, nops / ms / 1e6, nops * (double)G / ms / 1e6);
+         M, R, G, (unsigned long long)(bytes >> 20), (unsigned long long)nops, ms, nops / ms / 1e6, nops * (double)G / ms / 1e6);
 }
 
 template <bool RET>
@@ -116,11 +149,48 @@ int main() {
   printf("{\"kind\": \"copy\", \"array_MB\": %llu, \"ms\": %.4f, \"GB_s\": %.1f}\n", (unsigned long long)(big >> 20), cms,
          2.0 * big / cms / 1e6);
   const uint64_t nops = 1ull << 25;
-  read_case<16>(a, big, nops, sink, blocks);
-  read_case<32>(a, big, nops, sink, blocks);
-  read_case<64>(a, big, nops, sink, blocks);
-  read_case<128>(a, big, nops, sink, blocks);
-  read_case<64>(a, 64ull << 20, nops, sink, blocks);     // L2-resident for contrast
+  if (getenv("RB_LDMODES")) {                  // load-instruction variants of random 32/64-B reads
+    read_case<32, 4, 0>(a, big, nops, sink, blocks);
+    read_case<32, 4, 1>(a, big, nops, sink, blocks);
+    read_case<32, 4, 2>(a, big, nops, sink, blocks);
+    read_case<32, 4, 3>(a, big, nops, sink, blocks);
+    read_case<64, 4, 0>(a, big, nops, sink, blocks);
+    read_case<64, 4, 1>(a, big, nops, sink, blocks);
+    read_case<16, 4, 0>(a, big, nops, sink, blocks);
+    read_case<16, 4, 1>(a, big, nops, sink, blocks);
+    cudaError_t e = cudaDeviceSynchronize();
+    return e ? 1 : 0;
+  }
+  for (uint64_t mb : {64ull, 128ull, 256ull, 2048ull, 4096ull}) {
+    read_case<16>(a, mb << 20, nops, sink, blocks);
+    read_case<32>(a, mb << 20, nops, sink, blocks);
+    read_case<64>(a, mb << 20, nops, sink, blocks);
+    read_case<128>(a, mb << 20, nops, sink, blocks);
+  }
+  read_case<32, 8>(a, big, nops, sink, blocks);
+  read_case<64, 8>(a, big, nops, sink, blocks);
+  read_case<128, 8>(a, big, nops, sink, blocks);
+  // the L2 fetch granularity limit (a hint): does a random sector miss fetch 32, 64 or 128 B?
+  for (int gr : {32, 64, 128}) {
+    size_t before = 0, after = 0;
+    cudaDeviceGetLimit(&before, cudaLimitMaxL2FetchGranularity);
+    cudaDeviceSetLimit(cudaLimitMaxL2FetchGranularity, gr);
+    cudaDeviceGetLimit(&after, cudaLimitMaxL2FetchGranularity);
+    printf("{\"kind\": \"l2_fetch_granularity\", \"before\": %zu, \"set\": %d, \"after\": %zu}\n", before, gr, after);
+    read_case<32>(a, big, nops, sink, blocks);
+    read_case<64>(a, big, nops, sink, blocks);
+    read_case<16>(a, 128ull << 20, nops, sink, blocks);
+    atomic_case<true>((uint32_t *)a, 1024ull << 20, nops, (uint32_t *)sink, blocks);
+  }
+  cudaDeviceSetLimit(cudaLimitMaxL2FetchGranularity, 128);
+  for (uint64_t mb : {1024ull, 2048ull}) {
+    const float m64 = timeit([&] { k_line_rmw<64, 4><<<blocks, 256>>>(a, (mb << 20) / 64, nops, 3); });
+    const float m128 = timeit([&] { k_line_rmw<128, 4><<<blocks, 256>>>(a, (mb << 20) / 128, nops, 3); });
+    printf("{\"kind\": \"line_rmw\", \"granule_B\": 64, \"array_MB\": %llu, \"ops\": %llu, \"ms\": %.4f, \"Gops_s\": %.3f}\n",
+           (unsigned long long)mb, (unsigned long long)nops, m64, nops / m64 / 1e6);
+    printf("{\"kind\": \"line_rmw\", \"granule_B\": 128, \"array_MB\": %llu, \"ops\": %llu, \"ms\": %.4f, \"Gops_s\": %.3f}\n",
+           (unsigned long long)mb, (unsigned long long)nops, m128, nops / m128 / 1e6);
+  }
   for (uint64_t mb : {64ull, 128ull, 256ull, 1024ull, 4096ull}) {
     atomic_case<true>((uint32_t *)a, mb << 20, nops, (uint32_t *)sink, blocks);
     atomic_case<false>((uint32_t *)a, mb << 20, nops, (uint32_t *)sink, blocks);
