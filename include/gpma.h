@@ -119,6 +119,8 @@ typedef struct {
   uint64_t total_slots_rewritten;   /* sum of last_slots_rewritten                       */
   uint64_t total_windows_rewritten;
   uint64_t last_pending_level1;    /* updates the leaves rejected (climbing to level 1)   */
+  uint64_t last_levels_skipped;    /* levels a root-bound climb passed over (no window there
+                                      could accept: dead-level skip)           */
 } gpma_stats_t;
 
 /* Fill *cfg with the defaults above. */

@@ -9,6 +9,9 @@
 #include <chrono>
 #include <cstdio>
 #include <cstring>
+#include <mutex>
+#include <unordered_map>
+#include <vector>
 
 #include "gpma_internal.cuh"
 
@@ -29,6 +32,38 @@ struct DevPool {
   int handles = 0;
 };
 DevPool g_pools[64];
+
+// Blocks >= 1 MiB (store arrays, root-merge and level scratch) freed by the library are kept in a
+// per-device cache keyed by exact size and handed back to the next request of that size, with
+// an event ordering the reuse after the freeing stream's work.  The pool alone re-mapped
+// fragmented free memory for such requests with its reserved size unchanged: 140-510 ms for
+// one 0.5-2 GiB request in a resizing step (tools/resize_trace.py, GPMA_TRACE_ALLOC=1).
+// GPMA_BLOCK_CACHE=0 disables it.  The cache is emptied into the pool when an allocation
+// fails (then the request is retried) and trimmed with the pool on the last destroy.
+constexpr size_t BIG_BLOCK = 1u << 20;
+struct CachedBlock {
+  void *p;
+  size_t bytes;
+  cudaEvent_t ev;
+};
+std::vector<CachedBlock> g_cache[64];
+std::unordered_map<void *, size_t> g_big_sizes[64];    // live big blocks of the library pool
+bool block_cache_on() {
+  static const bool on = [] {
+    const char *e = getenv("GPMA_BLOCK_CACHE");
+    return !e || atoi(e) != 0;
+  }();
+  return on;
+}
+// free every cached block of the device to its pool (caller holds g_pool_mu)
+void cache_flush_locked(int dev, cudaStream_t s) {
+  for (CachedBlock &b : g_cache[dev & 63]) {
+    cudaStreamWaitEvent(s, b.ev, 0);
+    cudaEventDestroy(b.ev);
+    cudaFreeAsync(b.p, s);
+  }
+  g_cache[dev & 63].clear();
+}
 }  // namespace
 
 static cudaMemPool_t lib_pool(int dev) {
@@ -74,7 +109,21 @@ void pool_detach(gpma *g) {
     if (const char *e = getenv("GPMA_POOL_KEEP_MB")) keep = (size_t)atoll(e) << 20;
     else if (cudaMemGetInfo(&fr, &tot) == cudaSuccess) keep = tot / 4;
     cudaGetLastError();
-    cudaMemPoolTrimTo(P.pool, keep);                    // every block is free by now
+    // cached big blocks count against the budget: the largest go back first
+    std::vector<CachedBlock> &C = g_cache[g->device & 63];
+    std::sort(C.begin(), C.end(), [](const CachedBlock &a, const CachedBlock &b) { return a.bytes < b.bytes; });
+    size_t cached = 0;
+    for (const CachedBlock &b : C) cached += b.bytes;
+    while (!C.empty() && cached > keep) {
+      CachedBlock b = C.back();
+      C.pop_back();
+      cached -= b.bytes;
+      cudaStreamWaitEvent(g->st, b.ev, 0);
+      cudaEventDestroy(b.ev);
+      cudaFreeAsync(b.p, g->st);
+    }
+    cudaStreamSynchronize(g->st);
+    cudaMemPoolTrimTo(P.pool, keep - cached);          // every other block is free by now
   }
   g->pool_attached = false;
 }
@@ -97,10 +146,39 @@ cudaError_t dev_alloc(gpma *g, void **p, size_t bytes, cudaStream_t s) {
     e = *p ? cudaSuccess : cudaErrorMemoryAllocation;
   } else {
     cudaMemPool_t pool = lib_pool(g->device);
-    e = pool ? cudaMallocFromPoolAsync(p, bytes, pool, s) : cudaMallocAsync(p, bytes, s);
+    const bool big = pool && bytes >= BIG_BLOCK && block_cache_on();
+    e = cudaErrorMemoryAllocation;
+    if (big) {
+      std::lock_guard<std::mutex> lk(g_pool_mu);
+      std::vector<CachedBlock> &C = g_cache[g->device & 63];
+      for (size_t i = 0; i < C.size(); ++i)
+        if (C[i].bytes == bytes) {
+          *p = C[i].p;
+          cudaStreamWaitEvent(s, C[i].ev, 0);          // after the freeing stream's last use
+          cudaEventDestroy(C[i].ev);
+          C.erase(C.begin() + (long)i);
+          g_big_sizes[g->device & 63][*p] = bytes;
+          e = cudaSuccess;
+          break;
+        }
+    }
     if (e != cudaSuccess) {
-      cudaGetLastError();
-      *p = nullptr;
+      e = pool ? cudaMallocFromPoolAsync(p, bytes, pool, s) : cudaMallocAsync(p, bytes, s);
+      if (e != cudaSuccess && big) {                  // give the cached blocks back, retry once
+        cudaGetLastError();
+        {
+          std::lock_guard<std::mutex> lk(g_pool_mu);
+          cache_flush_locked(g->device, s);
+        }
+        e = cudaMallocFromPoolAsync(p, bytes, pool, s);
+      }
+      if (e != cudaSuccess) {
+        cudaGetLastError();
+        *p = nullptr;
+      } else if (big) {
+        std::lock_guard<std::mutex> lk(g_pool_mu);
+        g_big_sizes[g->device & 63][*p] = bytes;
+      }
     }
   }
   if (trace_alloc() && bytes >= (64u << 20)) {
@@ -122,6 +200,22 @@ void dev_free(gpma *g, void *p, cudaStream_t s) {
   if (g->alloc_fn) {
     if (g->free_fn) g->free_fn(p, (gpma_stream_t)s, g->alloc_ctx);
     return;
+  }
+  {
+    std::lock_guard<std::mutex> lk(g_pool_mu);
+    auto &M = g_big_sizes[g->device & 63];
+    auto it = M.find(p);
+    if (it != M.end()) {
+      CachedBlock b{p, it->second, nullptr};
+      M.erase(it);
+      if (cudaEventCreateWithFlags(&b.ev, cudaEventDisableTiming) == cudaSuccess &&
+          cudaEventRecord(b.ev, s) == cudaSuccess) {
+        g_cache[g->device & 63].push_back(b);
+        return;
+      }
+      cudaGetLastError();
+      if (b.ev) cudaEventDestroy(b.ev);
+    }
   }
   cudaFreeAsync(p, s);
 }

@@ -4343,6 +4343,80 @@ static gpma_status big_groups(gpma *g, const uint64_t *ik, const uint32_t *iv, u
   return GPMA_OK;
 }
 
+// ---- dead-level skip (exact).  A window's density-test value -- n_W + |U_W| for inserts,
+// n_W - |D_W| for strict deletes (Alg. 4 l.23-25) -- does not change when its sub-windows absorb
+// their updates at lower levels: absorbed updates move from pending to live (or leave both
+// counts).  So from the current leaf live counts and pending list, one pass finds the lowest level
+// in [lvl0, lvl1) at which some window holding pending updates would accept; the levels below it
+// change nothing (no window accepts, the pending list is carried up unchanged) and are skipped.
+// A root-bound climb (a resizing batch) then goes from the first empty level straight to the root.
+__global__ void k_set_u32(uint32_t *p, uint32_t v) { *p = v; }
+
+struct LvlBound {
+  uint64_t t[64];       // max_i (insert) or min_i (strict delete) per level
+};
+__global__ void k_lvl_first_accept(const uint32_t *__restrict__ pt, uint64_t p, const uint32_t *__restrict__ pre,
+                                   uint32_t lvl0, uint32_t lvl1, LvlBound tb, int op, uint32_t *first) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < p; i += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t t = pt[i];
+    const uint32_t tp = i ? pt[i - 1] : 0u;
+    uint64_t e = i + 1;                        // end of i's window at the level below (exclusive)
+    for (uint32_t j = lvl0; j < lvl1; ++j) {
+      if (j >= *(volatile uint32_t *)first) break;          // a lower accepting level is known
+      if (i && (tp >> j) == (t >> j)) break;                 // not the window's first update
+      const uint32_t w = t >> j;
+      uint64_t lo = e, hi = e, step = 1;                     // first index past the window
+      while (hi < p && (pt[hi] >> j) == w) {
+        lo = hi + 1;
+        hi += step;
+        step <<= 1;
+      }
+      if (hi > p) hi = p;
+      while (lo < hi) {
+        const uint64_t mid = (lo + hi) >> 1;
+        if ((pt[mid] >> j) == w) lo = mid + 1;
+        else hi = mid;
+      }
+      e = lo;
+      const uint64_t a0 = (uint64_t)w << j, a1 = (uint64_t)(w + 1) << j;
+      const uint64_t n = (uint64_t)(pre[a1] - pre[a0]);
+      const uint64_t u = e - i;
+      const bool ok = op == GPMA_INSERT ? n + u <= tb.t[j] : (n >= u && n - u >= tb.t[j]);
+      if (ok) {
+        atomicMin(first, j);
+        break;
+      }
+    }
+  }
+}
+
+// GPMA_LVL_SKIP=0 disables the dead-level skip (read per call)
+static bool lvl_skip_on() {
+  const char *e = getenv("GPMA_LVL_SKIP");
+  return !e || atoi(e) != 0;
+}
+constexpr uint64_t SKIP_MINP = 256;     // pending updates worth the prefix of the counts
+
+// the lowest level in [lvl0, lvl1) at which a window of the pending list (buffers cur) accepts,
+// lvl1 if none
+static gpma_status first_accept_level(gpma *g, int cur, uint64_t p, uint32_t lvl0, uint32_t lvl1, int op,
+                                      uint32_t *out, cudaStream_t s) {
+  const uint64_t nl = g->cap / g->L;
+  GP_CHECK(g, ensure(g, g->b_misc3, (nl + 2) * 4, s));
+  uint32_t *pre = (uint32_t *)g->b_misc3.p, *first = pre + nl + 1;
+  GP_CHECK(g, scan_u32(g, g->cnt, pre, nl, s));
+  GP_LAUNCH(g, k_set_u32, 1, 1, 0, s, first, lvl1);
+  LvlBound tb{};
+  const std::vector<uint64_t> &b = op == GPMA_INSERT ? g->tmax : g->tmin;
+  for (uint32_t j = 0; j < 64 && j < b.size(); ++j) tb.t[j] = b[j];
+  GP_LAUNCH(g, k_lvl_first_accept, grid_for(p), TB, 0, s, (const uint32_t *)g->b_pt[cur].p, p, pre, lvl0, lvl1, tb,
+            op, first);
+  GP_CHECK(g, readback(g, g->pin, first, 4, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  memcpy(out, g->pin, 4);
+  return GPMA_OK;
+}
+
 // After the prefix's host round trip: the pending list of level 1 (if any), the level loop, the
 // root resize, the head fix-up.  ik / iv: the batch the prefix read (staged or the caller's).
 static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int path,
@@ -4450,6 +4524,8 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     if ((st = coop_levels(g, cur, p, lvl, &dirty_base, op, s))) return st;
   }
   Nvtx nvtx_levels("update: host level loop");
+  const bool skip = lvl_skip_on() && !g->trace_on && g->cap < (1ull << 32) && g->h < 64;
+  uint32_t next_check = 0;
   for (; lvl <= g->h && p > 0; ++lvl) {
     Lvl a = make_lvl(g, cur, p, lvl, op);
     LevelOut lo{};
@@ -4458,7 +4534,18 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     g->last.last_windows_rewritten += lo.nacc;
     g->last.last_top_level = lvl;
     if (lo.p_new) cur ^= 1;
+    const uint64_t p_in = p;
     p = lo.p_new;
+    if (skip && p >= SKIP_MINP && 2 * p > p_in && lvl + 1 < g->h && lvl >= next_check) {
+      // a level that absorbed less than half of many pending updates: likely a root-bound climb
+      // -- jump over the levels where no window accepts (nothing happens there).  A check that
+      // finds the next level accepting backs off for two levels.
+      uint32_t j = 0;
+      if ((st = first_accept_level(g, cur, p, lvl + 1, g->h, op, &j, s))) return st;
+      g->last.last_levels_skipped += j - (lvl + 1);
+      if (j == lvl + 1) next_check = lvl + 3;
+      lvl = j - 1;
+    }
   }
   if (p > 0) {
     g->last.last_top_level = g->h + 1;

@@ -240,3 +240,42 @@ def test_oversized_leaf_groups(mode):
     _apply(g, o, ks[:8000], op=1)
     _apply(g, o, ks[4000:12000], vs[4000:12000])
     assert_same_csr(g, o)
+
+
+@pytest.mark.parametrize("mode", [0, 1])
+def test_dead_level_skip_intermediate_and_root(mode):
+    """The dead-level skip: a hot batch from a handful of rows climbs levels where its
+    one or two windows reject (nacc = 0 with >= 2^14 pending), so the skip jumps to the first level
+    whose window accepts (Alg. 4 l.23-25: n_W + |U_W| is unchanged by lower levels) -- the layout,
+    top level, windows and slots rewritten must equal both the oracle and the loop run level by
+    level (GPMA_LVL_SKIP=0).  Then strict deletes of the same keys climb the same way."""
+    import os
+    V = 1 << 12
+    rng = np.random.default_rng(5)
+    src = rng.integers(0, V, 1 << 17, dtype=np.uint64)
+    dst = rng.integers(0, V, 1 << 17, dtype=np.uint64)
+    k0 = np.unique((src << np.uint64(32)) | dst)
+    v0 = (np.arange(len(k0)) % 1000).astype(np.uint32)
+    hot = np.array([(np.uint64(7 + r) << np.uint64(32)) | np.uint64(c) for r in range(5) for c in range(V)],
+                   dtype=np.uint64)
+    hot = np.setdiff1d(hot, k0)[: 3 * (1 << 13)]                    # >= 2^14 new keys, 5 rows
+    hv = (np.arange(len(hot)) % 777).astype(np.uint32)
+    stats = []
+    for skip in ("1", "0"):
+        os.environ["GPMA_LVL_SKIP"] = skip
+        try:
+            g, o = _pair(V, k0, v0, delete_mode=mode)
+            _apply(g, o, hot, hv)
+            si = g.gpma_stats()
+            if mode == 1:
+                _apply(g, o, hot, op=1)
+            sd = g.gpma_stats()
+            stats.append((si, sd))
+        finally:
+            os.environ.pop("GPMA_LVL_SKIP", None)
+    (si1, sd1), (si0, sd0) = stats
+    keys = ("last_top_level", "last_windows_rewritten", "last_slots_rewritten", "capacity", "resizes")
+    assert {k: si1[k] for k in keys} == {k: si0[k] for k in keys}
+    assert {k: sd1[k] for k in keys} == {k: sd0[k] for k in keys}
+    assert si1["last_levels_skipped"] > 0 and si0["last_levels_skipped"] == 0
+    assert si1["last_top_level"] <= si1["height"], "the hot batch should be absorbed below the root"

@@ -27,7 +27,7 @@ def seq(a, b):
 
 
 s = torch.cuda.Stream(dev)
-for rep in range(int(sys.argv[1]) if len(sys.argv) > 1 else 3):
+for rep in range(int(sys.argv[1]) if len(sys.argv) > 1 else 3):  # noqa: C901
     f, b = 0, 1 << 23
     with torch.cuda.stream(s):
         k0, v0 = seq(f, b)
@@ -59,8 +59,9 @@ for rep in range(int(sys.argv[1]) if len(sys.argv) > 1 else 3):
                 res0 = st["resizes"]
                 ksum = sum(v[1] for v in prof.values())
                 print(f"rep {rep} step {step} cap {st['capacity']}: events {e0.elapsed_time(e1):.2f} ms, "
-                      f"wall insert {1e3 * (w1 - w0):.2f} delete {1e3 * (w2 - w1):.2f} ms, kernels {ksum:.2f} ms",
-                      flush=True)
+                      f"wall insert {1e3 * (w1 - w0):.2f} delete {1e3 * (w2 - w1):.2f} ms, kernels {ksum:.2f} ms "
+                      f"(levels skipped {st.get('last_levels_skipped', 0)} in the last call, top level "
+                      f"{st['last_top_level']})", flush=True)
                 for k, v in sorted(prof.items(), key=lambda kv: -kv[1][1])[:8]:
                     print(f"    {k:24s} {v[0]:4d} {v[1]:.3f}", flush=True)
         del g
