@@ -339,6 +339,7 @@ struct gpma {
   // store (HBM-resident)
   uint64_t *key = nullptr;        // [cap]
   uint32_t *val = nullptr;        // [cap]
+  bool root_heads_done = false;   // the last root re-layout wrote the locate heads
   uint32_t *cnt = nullptr;        // [3*cap/L]: live entries (incl. guards) per leaf, then the
                                   // per-leaf tombstone bit mask (bit p = slot p is a tombstone),
                                   // then the guards per leaf

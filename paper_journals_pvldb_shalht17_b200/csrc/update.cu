@@ -2804,16 +2804,19 @@ __global__ void __launch_bounds__(CL_T) k_levels_coop(CoopArgs a) {
 
 // Whole-array even layout of a dense sorted list (create, resize; R7 over all leaves): a thread
 // writes 4 consecutive slots of one leaf with 16-B stores (two key pairs, one value quad).
+// (head != nullptr: also the locate heads, valid when N >= nleaves -- then no leaf is empty and
+// head[l] is the leaf's first key; the caller recomputes them otherwise)
 __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *__restrict__ wv,
                               uint64_t N, uint64_t *__restrict__ key, uint32_t *__restrict__ val,
                               uint32_t *__restrict__ cnt, uint64_t *__restrict__ row_offset,
-                              uint32_t L, uint64_t nleaves, uint32_t rb) {
+                              uint32_t L, uint64_t nleaves, uint32_t rb, uint64_t *__restrict__ head) {
   uint32_t *tmask = cnt + nleaves;
   const uint64_t cap = nleaves * L;
+  const int lg = __ffsll((long long)nleaves) - 1;       // nleaves: a power of two
   for (uint64_t s = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) * 4; s < cap;
        s += (uint64_t)gridDim.x * blockDim.x * 4) {
     const uint64_t l = leaf_div(s, L), p = leaf_mod(s, L);
-    const uint64_t lo = l * N / nleaves, hi = (l + 1) * N / nleaves, m = hi - lo;
+    const uint64_t lo = (l * N) >> lg, hi = ((l + 1) * N) >> lg, m = hi - lo;
     uint64_t k[4];
     uint32_t v[4];
 #pragma unroll
@@ -2836,6 +2839,7 @@ __global__ void k_layout_even(const uint64_t *__restrict__ wk, const uint32_t *_
       uint32_t gc = 0;
       for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(wk[e]);
       tmask[nleaves + l] = gc;
+      if (head) head[l] = k[0];
     }
   }
 }
@@ -3080,10 +3084,12 @@ gpma_status build_from_sorted(gpma *g, const uint64_t *wk, const uint32_t *wv, u
                               cudaStream_t s) {
   uint64_t nl = g->cap / g->L;
   GP_LAUNCH(g, k_layout_even, grid_for(g->cap / 4), TB, 0, s, wk, wv, N, g->key, g->val, g->cnt,
-            g->row_offset, g->L, nl, g->rb);
+            g->row_offset, g->L, nl, g->rb, N >= nl ? g->head : nullptr);
   GP_CHECK(g, cudaGetLastError());
-  gpma_status st = recompute_heads(g, s);
-  if (st) return st;
+  if (N < nl) {
+    gpma_status st = recompute_heads(g, s);
+    if (st) return st;
+  }
   return recompute_degrees(g, s);
 }
 
@@ -3246,7 +3252,7 @@ static bool gather_big_on() {
 
 static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t *dirty_base,
                               cudaStream_t s, bool resize_target, uint64_t new_cap, uint64_t *nk,
-                              uint32_t *nv, uint32_t *ncnt) {
+                              uint32_t *nv, uint32_t *ncnt, uint64_t *nhead = nullptr) {
   const uint64_t p = a.p;
   const uint64_t nleaves = g->cap / g->L;
   const uint64_t wins_bound = std::min<uint64_t>(p, nleaves >> a.lvl);
@@ -3328,8 +3334,9 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
       GP_CHECK(g, cudaStreamSynchronize(s));
       N = g->ctrl_h->sum;
       uint64_t nl_new = new_cap / g->L;
+      g->root_heads_done = nhead && N >= nl_new;
       GP_LAUNCH(g, k_layout_even, grid_for(new_cap / 4), TB, 0, s, a.wk, a.wv, N, nk, nv, ncnt,
-                g->row_offset, g->L, nl_new, g->rb);
+                g->row_offset, g->L, nl_new, g->rb, g->root_heads_done ? nhead : nullptr);
     }
   }
   }
@@ -3491,7 +3498,8 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   a.force = 1;
   LevelOut lo{};
   g->root_need = ntot + p;                 // the dense root list: live entries + the pending
-  st = level_step(g, a, cur, &lo, dirty_base, s, true, cap, nk, nv, ncnt);
+  g->root_heads_done = false;
+  st = level_step(g, a, cur, &lo, dirty_base, s, true, cap, nk, nv, ncnt, nhead);
   g->root_need = 0;
   if (st) return st;
   tr.stamp("root_merge");
@@ -3515,7 +3523,7 @@ static gpma_status resize(gpma *g, int cur, uint64_t p, int op, cudaStream_t s, 
   set_geometry(g, cap);
   g->last.last_slots_rewritten += cap;
   g->last.last_windows_rewritten += 1;
-  st = recompute_heads(g, s);
+  st = g->root_heads_done ? GPMA_OK : recompute_heads(g, s);   // (heads written by the layout)
   tr.stamp("heads");
   return st;
 }
@@ -3735,8 +3743,9 @@ static gpma_status double_root(gpma *g, cudaStream_t s) {
   uint32_t *nv, *ncnt;
   uint64_t *nhead;
   if ((st = alloc_store(g, cap2, &nk, &nv, &ncnt, &nhead, s))) return st;
+  const bool heads_done = N >= cap2 / g->L;
   GP_LAUNCH(g, k_layout_even, grid_for(cap2 / 4), TB, 0, s, (const uint64_t *)g->b_wk.p, (const uint32_t *)g->b_wv.p,
-            N, nk, nv, ncnt, g->row_offset, g->L, cap2 / g->L, g->rb);
+            N, nk, nv, ncnt, g->row_offset, g->L, cap2 / g->L, g->rb, heads_done ? nhead : nullptr);
   if (spare_on()) {
     spare_stash(g, g->cap, g->key, g->val, g->cnt, g->head, s);
   } else {
@@ -3754,7 +3763,7 @@ static gpma_status double_root(gpma *g, cudaStream_t s) {
   set_geometry(g, cap2);
   g->last.last_slots_rewritten += cap2;
   g->last.last_windows_rewritten += 1;
-  return recompute_heads(g, s);
+  return heads_done ? GPMA_OK : recompute_heads(g, s);
 }
 
 __global__ void k_upd_summary(const uint32_t *__restrict__ pos, const uint32_t *__restrict__ kpos, uint64_t n,
