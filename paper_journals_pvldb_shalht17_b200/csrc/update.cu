@@ -4399,6 +4399,15 @@ __global__ void k_lvl_first_accept(const uint32_t *__restrict__ pt, uint64_t p, 
   }
 }
 
+// GPMA_TRACE_LEVELS=1: every host-driven level of a batch on stderr (diagnostics)
+static bool trace_levels() {
+  static const bool on = [] {
+    const char *e = getenv("GPMA_TRACE_LEVELS");
+    return e && atoi(e) != 0;
+  }();
+  return on;
+}
+
 // GPMA_LVL_SKIP=0 disables the dead-level skip (read per call)
 static bool lvl_skip_on() {
   const char *e = getenv("GPMA_LVL_SKIP");
@@ -4528,9 +4537,18 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     lvl = 1;
   }
   if (lvl == 1) g->last.last_pending_level1 = p;
+  if (trace_levels())
+    fprintf(stderr, "[gpma] prefix + level 0: %llu pending for level %u at %.3f ms\n", (unsigned long long)p, lvl,
+            std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - tl_call_start).count());
   if (p > 0 && lvl >= 1 && lvl <= g->h && !g->trace_on && coop_eligible(g, p, lvl)) {
     Nvtx nv("update: device level loop");
+    const uint64_t p0 = p;
+    const uint32_t l0 = lvl;
     if ((st = coop_levels(g, cur, p, lvl, &dirty_base, op, s))) return st;
+    if (trace_levels())
+      fprintf(stderr, "[gpma] device level loop %u..%u  pending %llu -> %llu  at %.3f ms\n", l0, lvl - 1,
+              (unsigned long long)p0, (unsigned long long)p,
+              std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - tl_call_start).count());
   }
   Nvtx nvtx_levels("update: host level loop");
   const bool skip = lvl_skip_on() && !g->trace_on && g->cap < (1ull << 32) && g->h < 64;
@@ -4545,6 +4563,10 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     if (lo.p_new) cur ^= 1;
     const uint64_t p_in = p;
     p = lo.p_new;
+    if (trace_levels())                                   // (level_step ended on a stream sync)
+      fprintf(stderr, "[gpma] level %2u  pending %9llu -> %9llu  accepted %8llu  at %.3f ms\n", lvl,
+              (unsigned long long)p_in, (unsigned long long)p, (unsigned long long)lo.nacc,
+              std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - tl_call_start).count());
     if (skip && p >= SKIP_MINP && 2 * p > p_in && lvl + 1 < g->h && lvl >= next_check) {
       // a level that absorbed less than half of many pending updates: likely a root-bound climb
       // -- jump over the levels where no window accepts (nothing happens there).  A check that
