@@ -689,6 +689,98 @@ __global__ void k_gflags(const uint64_t *__restrict__ tk, uint64_t n, uint32_t *
     hf[i] = (i == 0 || tk[i] != tk[i - 1]) ? 1u : 0u;
 }
 
+// Group starts of the leaf-sorted batch in ONE pass (UniqueSegments, Alg. 4 l.18-21, for level
+// 0): a decoupled look-back compaction of the head flags (tk[j] != tk[j-1]) -- gstart[g] = first
+// index of group g, gstart[ng] = n, *ng_out = ng.  Replaces flags + scan + scatter (three passes
+// over the batch and two launches more).  status[0] is the tile counter, status[1 + t] tile t's
+// (flag:2 | count) word; the caller zeroes both.
+constexpr int GS_T = 256, GS_I = 16, GS_TILE = GS_T * GS_I;
+__global__ void __launch_bounds__(GS_T) k_group_starts(const uint64_t *__restrict__ tk, uint64_t n,
+                                                       uint32_t *__restrict__ gstart, uint32_t *__restrict__ ng_out,
+                                                       unsigned long long *status, const Ctrl *c) {
+  __shared__ uint32_t s_tile, s_prefix;
+  __shared__ uint32_t wcnt[GS_T / 32];
+  if (c->err) return;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  if (threadIdx.x == 0) s_tile = (uint32_t)atomicAdd(status, 1ull);
+  __syncthreads();
+  const uint32_t tile = s_tile;
+  volatile unsigned long long *st = status + 1;
+  const uint64_t base = (uint64_t)tile * GS_TILE + (uint64_t)w * (32 * GS_I);
+  uint32_t bal[GS_I];
+  uint32_t mine = 0;
+#pragma unroll
+  for (int j = 0; j < GS_I; ++j) {
+    const uint64_t i = base + j * 32 + lane;
+    const bool f = i < n && (i == 0 || tk[i] != tk[i - 1]);
+    bal[j] = __ballot_sync(0xffffffffu, f);
+    mine += __popc(bal[j]);
+  }
+  if (lane == 0) wcnt[w] = mine;
+  __syncthreads();
+  if (w == 0) {
+    const uint32_t wc = lane < GS_T / 32 ? wcnt[lane] : 0u;
+    uint32_t x = wc;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+      if (lane >= o) x += y;
+    }
+    const uint32_t agg = __shfl_sync(0xffffffffu, x, 31);
+    if (lane < GS_T / 32) wcnt[lane] = x - wc;          // warp offsets inside the tile
+    const unsigned long long VMASK = (1ull << 62) - 1;
+    if (lane == 0) {
+      __threadfence();
+      st[tile] = ((tile == 0 ? 2ull : 1ull) << 62) | (unsigned long long)agg;
+    }
+    uint64_t prefix = 0;
+    for (int64_t t = (int64_t)tile - 1; t >= 0; t -= 32) {   // warp-parallel look-back
+      const int64_t q = t - lane;
+      unsigned long long v = 2ull << 62;
+      if (q >= 0) {
+        do { v = st[q]; } while ((v >> 62) == 0);
+      }
+      const uint32_t inc = __ballot_sync(0xffffffffu, (v >> 62) == 2);
+      const int stop = inc ? __ffs(inc) - 1 : 31;
+      uint64_t contrib = lane <= stop ? (v & VMASK) : 0ull;
+      for (int o = 16; o; o >>= 1) contrib += __shfl_xor_sync(0xffffffffu, contrib, o);
+      prefix += contrib;
+      if (inc) break;
+    }
+    if (lane == 0) {
+      if (tile) {
+        __threadfence();
+        st[tile] = (2ull << 62) | (unsigned long long)(prefix + agg);
+      }
+      s_prefix = (uint32_t)prefix;
+      if ((uint64_t)(tile + 1) * GS_TILE >= n) {        // last tile: the end sentinel and the count
+        gstart[prefix + agg] = (uint32_t)n;
+        *ng_out = (uint32_t)(prefix + agg);
+      }
+    }
+  }
+  __syncthreads();
+  uint32_t r = s_prefix + wcnt[w];
+  const uint32_t lt = (1u << lane) - 1u;
+#pragma unroll
+  for (int j = 0; j < GS_I; ++j) {
+    if ((bal[j] >> lane) & 1u) gstart[r + __popc(bal[j] & lt)] = (uint32_t)(base + j * 32 + lane);
+    r += __popc(bal[j]);
+  }
+}
+
+static gpma_status group_starts(gpma *g, const uint64_t *tk, uint64_t n, uint32_t *gstart, uint32_t *ng_out,
+                                cudaStream_t s) {
+  const uint64_t nt = std::max<uint64_t>(1, (n + GS_TILE - 1) / GS_TILE);
+  DevBuf &sb = tl_scan ? *tl_scan : g->b_scan;
+  GP_CHECK(g, ensure(g, sb, (nt + 1) * sizeof(unsigned long long), s));
+  GP_CHECK(g, fill_zero(g, sb.p, (nt + 1) * sizeof(unsigned long long), s));
+  GP_LAUNCH(g, k_group_starts, (unsigned)nt, GS_T, 0, s, tk, n, gstart, ng_out, (unsigned long long *)sb.p,
+            g->ctrl_d);
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 // One thread per leaf group of the leaf-sorted batch (updates in arrival order): the leaf in
 // registers as in k_ins_leaf_t.  Pass 1 decides every update -- a later copy of the same key in
 // the group supersedes it (R10); a key equal to an occupied slot overwrites / revives it
@@ -3898,6 +3990,12 @@ static float interp_fv(gpma *g) {
   return 1.0f / (float)std::max<uint32_t>(g->V, 1u);
 }
 
+// GPMA_GSTART_FUSED=0: group starts by flags + scan + scatter (read per call)
+static bool gstart_fused() {
+  const char *e = getenv("GPMA_GSTART_FUSED");
+  return !e || atoi(e) != 0;
+}
+
 static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, int op, Sorted *srt,
                               cudaStream_t s) {
   gpma_status st;
@@ -3949,10 +4047,15 @@ static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, i
     const uint32_t *tix = which ? tx1 : tx0;
     srt->k = (uint64_t *)tk;
     srt->v = (uint32_t *)tix;
-    uint32_t *hf = keep2, *gid = kpos, *gstart = (uint32_t *)g->b_wfirst.p;
-    GP_LAUNCH(g, k_gflags, grid_for(n), TB, 0, s, tk, n, hf, g->ctrl_d);
-    GP_CHECK(g, scan_u32(g, hf, gid, n, s));
-    GP_LAUNCH(g, k_gstart, grid_for(n), TB, 0, s, hf, gid, n, gstart, g->ctrl_d);
+    uint32_t *gid = kpos, *gstart = (uint32_t *)g->b_wfirst.p;
+    if (gstart_fused()) {
+      if ((st = group_starts(g, tk, n, gstart, gid + n, s))) return st;
+    } else {
+      uint32_t *hf = keep2;
+      GP_LAUNCH(g, k_gflags, grid_for(n), TB, 0, s, tk, n, hf, g->ctrl_d);
+      GP_CHECK(g, scan_u32(g, hf, gid, n, s));
+      GP_LAUNCH(g, k_gstart, grid_for(n), TB, 0, s, hf, gid, n, gstart, g->ctrl_d);
+    }
     const uint32_t bound = (uint32_t)g->tmax[0];
     uint2 *dirty = (uint2 *)g->b_dirty.p;
     GP_CHECK(g, ensure(g, g->b_tgt, (n + 1) * 4, s));
