@@ -33,20 +33,36 @@ struct DevPool {
 };
 DevPool g_pools[64];
 
-// Blocks >= 1 MiB (store arrays, root-merge and level scratch) freed by the library are kept in a
+// Blocks >= 64 MiB (store arrays, root-merge and level scratch) freed by the library are kept in a
 // per-device cache keyed by exact size and handed back to the next request of that size, with
 // an event ordering the reuse after the freeing stream's work.  The pool alone re-mapped
 // fragmented free memory for such requests with its reserved size unchanged: 140-510 ms for
 // one 0.5-2 GiB request in a resizing step (tools/resize_trace.py, GPMA_TRACE_ALLOC=1).
 // GPMA_BLOCK_CACHE=0 disables it.  The cache is emptied into the pool when an allocation
 // fails (then the request is retried) and trimmed with the pool on the last destroy.
-constexpr size_t BIG_BLOCK = 1u << 20;
+constexpr size_t BIG_BLOCK = 64u << 20;
 struct CachedBlock {
   void *p;
   size_t bytes;
   cudaEvent_t ev;
 };
-std::vector<CachedBlock> g_cache[64];
+std::vector<CachedBlock> g_cache[64];                 // oldest first
+size_t g_cache_bytes[64];
+// bytes the cache may hold per device (GPMA_BLOCK_CACHE_MB, default an eighth of the device):
+// beyond it the oldest blocks go back to the pool
+size_t cache_limit(int dev) {
+  static size_t lim[64];
+  size_t &l = lim[dev & 63];
+  if (!l) {
+    size_t fr = 0, tot = 0;
+    if (const char *e = getenv("GPMA_BLOCK_CACHE_MB")) l = (size_t)atoll(e) << 20;
+    else if (cudaMemGetInfo(&fr, &tot) == cudaSuccess) l = tot / 8;
+    else l = (size_t)8 << 30;
+    cudaGetLastError();
+    if (!l) l = 1;
+  }
+  return l;
+}
 std::unordered_map<void *, size_t> g_big_sizes[64];    // live big blocks of the library pool
 bool block_cache_on() {
   static const bool on = [] {
@@ -63,6 +79,7 @@ void cache_flush_locked(int dev, cudaStream_t s) {
     cudaFreeAsync(b.p, s);
   }
   g_cache[dev & 63].clear();
+  g_cache_bytes[dev & 63] = 0;
 }
 }  // namespace
 
@@ -118,6 +135,7 @@ void pool_detach(gpma *g) {
       CachedBlock b = C.back();
       C.pop_back();
       cached -= b.bytes;
+      g_cache_bytes[g->device & 63] -= b.bytes;
       cudaStreamWaitEvent(g->st, b.ev, 0);
       cudaEventDestroy(b.ev);
       cudaFreeAsync(b.p, g->st);
@@ -156,6 +174,7 @@ cudaError_t dev_alloc(gpma *g, void **p, size_t bytes, cudaStream_t s) {
           *p = C[i].p;
           cudaStreamWaitEvent(s, C[i].ev, 0);          // after the freeing stream's last use
           cudaEventDestroy(C[i].ev);
+          g_cache_bytes[g->device & 63] -= C[i].bytes;
           C.erase(C.begin() + (long)i);
           g_big_sizes[g->device & 63][*p] = bytes;
           e = cudaSuccess;
@@ -210,7 +229,19 @@ void dev_free(gpma *g, void *p, cudaStream_t s) {
       M.erase(it);
       if (cudaEventCreateWithFlags(&b.ev, cudaEventDisableTiming) == cudaSuccess &&
           cudaEventRecord(b.ev, s) == cudaSuccess) {
-        g_cache[g->device & 63].push_back(b);
+        std::vector<CachedBlock> &C = g_cache[g->device & 63];
+        size_t &cb = g_cache_bytes[g->device & 63];
+        C.push_back(b);
+        cb += b.bytes;
+        const size_t lim = cache_limit(g->device);
+        while (cb > lim && C.size() > 1) {             // the oldest go back to the pool
+          CachedBlock o = C.front();
+          C.erase(C.begin());
+          cb -= o.bytes;
+          cudaStreamWaitEvent(s, o.ev, 0);
+          cudaEventDestroy(o.ev);
+          cudaFreeAsync(o.p, s);
+        }
         return;
       }
       cudaGetLastError();
