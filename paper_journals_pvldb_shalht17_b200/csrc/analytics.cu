@@ -1278,13 +1278,6 @@ gpma_status pagerank_f32(gpma *g, float *x, int warm, float d, float tol, int ma
 
 // ------------------------------------------------------------------ export CSR
 // edges per leaf = live entries - guards (both maintained per leaf by every rewrite)
-__global__ void k_exp_counts(const uint32_t *__restrict__ cnt, const uint32_t *__restrict__ gl, uint64_t nl,
-                             uint64_t *__restrict__ lc) {
-  for (uint64_t l = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; l < nl;
-       l += (uint64_t)gridDim.x * blockDim.x)
-    lc[l] = cnt[l] - gl[l];
-}
-
 // Compaction sweep, 4 slots per thread.  A warp's 128 slots are leaf aligned and their
 // edges land contiguously in the output from lbase[first leaf]: ranks come from a warp scan,
 // the (col, val) pairs are staged in shared memory and stored as full coalesced lines.
@@ -1417,8 +1410,7 @@ gpma_status export_csr(gpma *g, uint64_t *row_ptr, uint32_t *col, uint32_t *val,
   const uint64_t nl = g->cap / g->L;
   GP_CHECK(g, ensure(g, X.lpre, (nl + 1) * 8, s));
   uint64_t *lc = (uint64_t *)X.lpre.p;
-  GP_LAUNCH(g, k_exp_counts, grid_for(nl), TA, 0, s, g->cnt, gcnt_of(g), nl, lc);
-  GP_CHECK(g, scan_u64(g, lc, lc, nl, s));
+  GP_CHECK(g, scan_leaf_edges(g, g->cnt, gcnt_of(g), lc, nl, s));   // live edges per leaf, scanned
   GP_CHECK(g, readback(g, &X.ctrl_h->sum, lc + nl, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
   uint64_t nnz = X.ctrl_h->sum;

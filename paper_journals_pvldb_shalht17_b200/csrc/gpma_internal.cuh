@@ -447,6 +447,9 @@ void release(gpma *g, DevBuf &b, cudaStream_t s);
 // exclusive scan: out[0..n) = prefix sums of in[0..n), out[n] = total.  in == out allowed.
 [[nodiscard]] cudaError_t scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s);
 [[nodiscard]] cudaError_t scan_u64(gpma *g, const uint64_t *in, uint64_t *out, uint64_t n, cudaStream_t s);
+// exclusive scan of (cnt[l] - gl[l]) over l < nl into out[0..nl] (the export's leaf offsets)
+[[nodiscard]] cudaError_t scan_leaf_edges(gpma *g, const uint32_t *cnt, const uint32_t *gl, uint64_t *out, uint64_t nl,
+                                          cudaStream_t s);
 // stable onesweep LSD radix sort of (key, val) pairs (vals may be null: keys only) on the
 // given 8-bit digit shifts; *which = the index (0/1) of the buffer pair holding the result.
 [[nodiscard]] cudaError_t radix_sort_pairs(gpma *g, uint64_t *k0, uint32_t *v0, uint64_t *k1, uint32_t *v1,

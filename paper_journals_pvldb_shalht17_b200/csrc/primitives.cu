@@ -477,17 +477,21 @@ int key_shifts(uint32_t V, int *shifts) {
 constexpr int SC_THREADS = 256;
 constexpr int SC_ITEMS = 16;
 constexpr int SC_TILE = SC_THREADS * SC_ITEMS;   // 4096
+// Scans of >= 2^22 items use 16K-item tiles: the look-back's inclusive prefix advances one
+// 32-tile window per L2 round trip, so 4K-item tiles put ~128 round trips on the critical path
+// of a 2^24-item scan (the export's leaf offsets: 107 us, 1.6 TB/s); small scans keep 4K tiles
+// (more CTAs, measured faster for the BFS / level-loop sizes).
+constexpr int SC_BIG_THREADS = 1024;
+constexpr uint64_t SC_BIG_MIN = 1ull << 22;
 
 template <typename T>
 __device__ __forceinline__ T warp_sum(T x) {
-#pragma unroll
   for (int o = 16; o; o >>= 1) x += __shfl_xor_sync(0xffffffffu, x, o);
   return x;
 }
 
 template <typename T>
 __device__ __forceinline__ T warp_incl_scan(T x, int lane) {
-#pragma unroll
   for (int o = 1; o < 32; o <<= 1) {
     T y = __shfl_up_sync(0xffffffffu, x, o);
     if (lane >= o) x += y;
@@ -495,28 +499,35 @@ __device__ __forceinline__ T warp_incl_scan(T x, int lane) {
   return x;
 }
 
-// Single-pass scan with decoupled look-back: each CTA takes the next tile id from a
-// counter, publishes its aggregate, then walks back over its predecessors' published
-// (aggregate | inclusive) values until it meets an inclusive prefix.  Status word:
-// flag in bits 62-63 (0 = not ready, 1 = aggregate, 2 = inclusive), value below.
 template <typename T>
-__global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *out, uint64_t n,
-                                                               unsigned long long *status) {
+struct ScanIn {                     // the plain input array
+  const T *in;
+  __device__ __forceinline__ T operator()(uint64_t i) const { return in[i]; }
+};
+
+// Single-pass exclusive scan with decoupled look-back (Merrill & Garland): each CTA takes the
+// next tile (atomic counter), publishes its aggregate, then sums predecessors' published
+// values back to the first inclusive prefix.  out[n] = total.  Status words live in
+// `status` (zeroed by the caller): [flag:2 | value:62], flag 1 = aggregate, 2 = inclusive.
+// In(i) yields item i (i < n), so producers can be fused into the scan.
+template <typename T, int NT, class In>
+__global__ void __launch_bounds__(NT) k_scan_lookback(In in, T *out, uint64_t n, unsigned long long *status) {
+  constexpr int TILE = NT * SC_ITEMS;
   __shared__ uint32_t s_tile;
-  __shared__ T ws[SC_THREADS / 32];
+  __shared__ T ws[NT / 32];
   __shared__ T s_prefix;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   if (threadIdx.x == 0) s_tile = status ? (uint32_t)atomicAdd(status, 1ull) : 0u;  // status[0] = tile counter
   __syncthreads();
   const uint32_t tile = s_tile;
   volatile unsigned long long *st = status ? status + 1 : nullptr;   // null: single tile
-  const uint64_t base = (uint64_t)tile * SC_TILE + (uint64_t)w * (32 * SC_ITEMS);
+  const uint64_t base = (uint64_t)tile * TILE + (uint64_t)w * (32 * SC_ITEMS);
   T x[SC_ITEMS];
   T part = 0;
 #pragma unroll
   for (int j = 0; j < SC_ITEMS; ++j) {
     uint64_t i = base + j * 32 + lane;
-    x[j] = i < n ? in[i] : T(0);
+    x[j] = i < n ? in(i) : T(0);
     part += x[j];
   }
   T wtot = warp_sum(part);
@@ -524,7 +535,7 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
   __syncthreads();
   if (w == 0) {
     T agg = 0;
-    for (int k = 0; k < SC_THREADS / 32; ++k) agg += ws[k];
+    for (int k = 0; k < NT / 32; ++k) agg += ws[k];
     const unsigned long long VMASK = (1ull << 62) - 1;
     T prefix = 0;
     if (lane == 0 && st) {
@@ -552,7 +563,7 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
         st[tile] = (2ull << 62) | ((unsigned long long)(prefix + agg) & VMASK);
       }
       s_prefix = prefix;
-      if ((uint64_t)(tile + 1) * SC_TILE >= n) out[n] = prefix + agg;   // last tile: total
+      if ((uint64_t)(tile + 1) * TILE >= n) out[n] = prefix + agg;   // last tile: total
     }
   }
   __syncthreads();
@@ -567,11 +578,14 @@ __global__ void __launch_bounds__(SC_THREADS) k_scan_lookback(const T *in, T *ou
   }
 }
 
-template <typename T>
-static cudaError_t scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) {
-  const uint64_t nt = (n + SC_TILE - 1) / SC_TILE > 0 ? (n + SC_TILE - 1) / SC_TILE : 1;
+template <typename T, class In>
+static cudaError_t scan_fn(gpma *g, const In &in, T *out, uint64_t n, cudaStream_t s) {
+  const bool big = n >= SC_BIG_MIN;
+  const uint64_t tile = big ? (uint64_t)SC_BIG_THREADS * SC_ITEMS : (uint64_t)SC_TILE;
+  const uint64_t nt = (n + tile - 1) / tile > 0 ? (n + tile - 1) / tile : 1;
   if (nt == 1) {                       // one tile: no look-back, no status reset
-    GP_LAUNCH(g, k_scan_lookback<T>, 1, SC_THREADS, 0, s, in, out, n, (unsigned long long *)nullptr);
+    GP_LAUNCH(g, (k_scan_lookback<T, SC_THREADS, In>), 1, SC_THREADS, 0, s, in, out, n,
+              (unsigned long long *)nullptr);
     return cudaGetLastError();
   }
   DevBuf &sb = tl_scan ? *tl_scan : g->b_scan;
@@ -579,8 +593,26 @@ static cudaError_t scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStrea
   if (e != cudaSuccess) return e;
   unsigned long long *status = (unsigned long long *)sb.p;
   if ((e = fill_zero(g, status, (nt + 1) * sizeof(unsigned long long), s)) != cudaSuccess) return e;
-  GP_LAUNCH(g, k_scan_lookback<T>, (unsigned)nt, SC_THREADS, 0, s, in, out, n, status);
+  if (big)
+    GP_LAUNCH(g, (k_scan_lookback<T, SC_BIG_THREADS, In>), (unsigned)nt, SC_BIG_THREADS, 0, s, in, out, n, status);
+  else
+    GP_LAUNCH(g, (k_scan_lookback<T, SC_THREADS, In>), (unsigned)nt, SC_THREADS, 0, s, in, out, n, status);
   return cudaGetLastError();
+}
+
+template <typename T>
+static cudaError_t scan_impl(gpma *g, const T *in, T *out, uint64_t n, cudaStream_t s) {
+  return scan_fn<T>(g, ScanIn<T>{in}, out, n, s);
+}
+
+// live edges per leaf (live count minus guards), scanned: the export's per-leaf output offsets
+struct LeafEdges {
+  const uint32_t *cnt, *gl;
+  __device__ __forceinline__ uint64_t operator()(uint64_t l) const { return (uint64_t)(cnt[l] - gl[l]); }
+};
+cudaError_t scan_leaf_edges(gpma *g, const uint32_t *cnt, const uint32_t *gl, uint64_t *out, uint64_t nl,
+                            cudaStream_t s) {
+  return scan_fn<uint64_t>(g, LeafEdges{cnt, gl}, out, nl, s);
 }
 
 cudaError_t scan_u32(gpma *g, const uint32_t *in, uint32_t *out, uint64_t n, cudaStream_t s) {

@@ -694,7 +694,7 @@ __global__ void k_gflags(const uint64_t *__restrict__ tk, uint64_t n, uint32_t *
 // index of group g, gstart[ng] = n, *ng_out = ng.  Replaces flags + scan + scatter (three passes
 // over the batch and two launches more).  status[0] is the tile counter, status[1 + t] tile t's
 // (flag:2 | count) word; the caller zeroes both.
-constexpr int GS_T = 256, GS_I = 16, GS_TILE = GS_T * GS_I;
+constexpr int GS_T = 1024, GS_I = 16, GS_TILE = GS_T * GS_I;   // 16K-item tiles: fewer look-back rounds
 __global__ void __launch_bounds__(GS_T) k_group_starts(const uint64_t *__restrict__ tk, uint64_t n,
                                                        uint32_t *__restrict__ gstart, uint32_t *__restrict__ ng_out,
                                                        unsigned long long *status, const Ctrl *c) {
