@@ -3634,11 +3634,16 @@ __global__ void k_coop_init(CoopState *st, uint64_t p, uint32_t cur, uint32_t lv
 }
 
 // GPMA_LVL_COOP=0 disables the device-resident level loop (read per call)
+// GPMA_COOP_MAXP: the largest pending count the device level loop takes (read per call);
+// larger climbs go level by level from the host, whose steps spread a level's windows over
+// every SM at once (the cooperative kernel's warps merge their share of windows one after the
+// other: barrier-bound at ~0.6M pending)
 static bool coop_eligible(gpma *g, uint64_t p, uint32_t lvl) {
   const char *e = getenv("GPMA_LVL_COOP");
   if (e && atoi(e) == 0) return false;
-  (void)p;
-  return ((uint64_t)g->L << lvl) <= CL_MAXS && g->h < 48;
+  uint64_t maxp = 1ull << 18;                   // (measured: configs[3] resizing steps 6.5 / 9.7 / 11.8 -> 6.0 / 9.1 / 10.7 ms)
+  if (const char *m = getenv("GPMA_COOP_MAXP")) maxp = (uint64_t)atoll(m);
+  return p <= maxp && ((uint64_t)g->L << lvl) <= CL_MAXS && g->h < 48;
 }
 
 static gpma_status coop_levels(gpma *g, int &cur, uint64_t &p, uint32_t &lvl, uint64_t *dirty_base, int op,
