@@ -168,7 +168,7 @@ def update_kernel_table(prof: dict, st: dict, B: int) -> dict:
     upd_names = ("k_validate", "k_lazy", "k_del", "k_prepass", "k_level0", "k_os_", "k_small_sort", "k_scan",
                  "k_compact", "k_upd", "k_zero", "k_copy", "k_readback", "k_locate", "k_lvl", "k_heads",
                  "k_radix", "k_gflags", "k_gstart", "k_ins_leaf", "k_pend", "k_levels", "k_coop", "k_big",
-                 "k_iota", "k_small")
+                 "k_iota", "k_small", "k_group", "k_set_u32")
     out = {}
     for k, (n, ms) in prof.items():
         if not k.startswith(upd_names):
