@@ -152,6 +152,9 @@ def update_roofline(st0: dict, st1: dict, slide_ms, B: int) -> dict:
             "formula": "12*n_ins + 8*n_del + 24*sum|W| + n_del_lazy*(8L+4) + 8*leaves_rewritten (SURVEY 8(d))"}
 
 
+RANDOM_CEILING_GBS = 5100.0   # DRAM traffic of independent random line fetches (profiles/random_access/)
+
+
 def update_kernel_table(prof: dict, st: dict, B: int) -> dict:
     """Per-kernel times of the update path in one profiled warm step (plain launches, no graph
     replay), with the algorithmic bytes SURVEY §8(d) assigns to the kernels that do the
@@ -159,6 +162,10 @@ def update_kernel_table(prof: dict, st: dict, B: int) -> dict:
     (fused level 0) 24·L per absorbed leaf + 12 per update; the existence pre-pass 12 + 8L per
     update.  Sort / scan / compaction kernels move implementation bytes only (no frac)."""
     hbm, _ = peaks()
+    try:
+        traffic = json.load(open(os.path.join(ROOT, "profiles", "ncu_traffic.json")))["dram_bytes_per_launch"]
+    except (OSError, ValueError, KeyError):
+        traffic = {}
     L = st["leaf_slots"]
     w0 = st.get("last_level0_windows", 0)
     leaf = 24 * L * w0 + 12 * B       # every absorbed leaf read + written, the batch read
@@ -178,6 +185,14 @@ def update_kernel_table(prof: dict, st: dict, B: int) -> dict:
             e["algorithmic_bytes"] = algo[k]
             e["achieved_gbs"] = algo[k] / (ms / 1e3) / 1e9
             e["frac"] = e["achieved_gbs"] / hbm
+        if k in traffic and ms > 0:
+            # ncu DRAM traffic per launch (profiles/ncu_traffic.json) over this run's time: the
+            # kernel's HBM GB/s, against the copy peak and the random-access ceiling (every
+            # random miss moves a 128-B line: ~40 G lines/s, profiles/random_access/)
+            e["dram_bytes_ncu"] = traffic[k]
+            e["dram_gbs"] = traffic[k] * n / (ms / 1e3) / 1e9
+            e["dram_frac_of_peak"] = e["dram_gbs"] / hbm
+            e["dram_frac_of_random_ceiling"] = e["dram_gbs"] / RANDOM_CEILING_GBS
         out[k] = e
     return dict(sorted(out.items(), key=lambda kv: -kv[1]["ms"]))
 

@@ -707,12 +707,25 @@ __global__ void __launch_bounds__(GS_T) k_group_starts(const uint64_t *__restric
   const uint32_t tile = s_tile;
   volatile unsigned long long *st = status + 1;
   const uint64_t base = (uint64_t)tile * GS_TILE + (uint64_t)w * (32 * GS_I);
-  uint32_t bal[GS_I];
-  uint32_t mine = 0;
+  // all of the warp's loads first (the flag's left neighbour comes from the next lane down,
+  // or from the previous row's lane 31; one extra load per warp)
+  uint64_t a[GS_I];
 #pragma unroll
   for (int j = 0; j < GS_I; ++j) {
     const uint64_t i = base + j * 32 + lane;
-    const bool f = i < n && (i == 0 || tk[i] != tk[i - 1]);
+    a[j] = i < n ? tk[i] : 0ull;
+  }
+  const uint64_t before = (lane == 0 && base > 0 && base <= n) ? tk[base - 1] : 0ull;
+  uint32_t bal[GS_I];
+  uint32_t mine = 0;
+  uint64_t carry = __shfl_sync(0xffffffffu, before, 0);
+#pragma unroll
+  for (int j = 0; j < GS_I; ++j) {
+    const uint64_t i = base + j * 32 + lane;
+    uint64_t left = __shfl_up_sync(0xffffffffu, a[j], 1);
+    if (lane == 0) left = carry;
+    carry = __shfl_sync(0xffffffffu, a[j], 31);
+    const bool f = i < n && (i == 0 || a[j] != left);
     bal[j] = __ballot_sync(0xffffffffu, f);
     mine += __popc(bal[j]);
   }
