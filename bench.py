@@ -612,6 +612,9 @@ def resize_stress(dev, grow_steps=242, shrink_steps=248):
             "ms_resize_step_mean": float(t[rz].mean()) if rz.any() else None,
             "ms_resize_steps": [round(float(x), 3) for x in t[rz]],
             "ms_other_step_mean": float(t[~rz].mean()),
+            "ms_other_step_p50_p99_max": [float(np.percentile(t[~rz], 50)), float(np.percentile(t[~rz], 99)),
+                                          float(t[~rz].max())],
+            "slowest_steps": [[int(i), float(t[i])] for i in np.argsort(-t)[:6]],
             "capacity_steps_up": dbl, "capacity_steps_down": hlv,
             "capacity": {"start": cap0, "max": max(caps), "end": caps[-1]}, "live_end": live,
             "setup_s": {"generate": gen_s}}

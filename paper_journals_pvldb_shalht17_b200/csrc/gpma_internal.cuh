@@ -8,6 +8,7 @@
 #include <atomic>
 #include <mutex>
 #include <string>
+#include <array>
 #include <vector>
 
 #include <nvtx3/nvToolsExt.h>
@@ -340,6 +341,7 @@ struct gpma {
   uint64_t *key = nullptr;        // [cap]
   uint32_t *val = nullptr;        // [cap]
   bool root_heads_done = false;   // the last root re-layout wrote the locate heads
+  std::vector<std::array<uint64_t, 3>> big_dirty;   // (first dirty entry, windows, leaves each) of big rewritten windows
   uint32_t *cnt = nullptr;        // [3*cap/L]: live entries (incl. guards) per leaf, then the
                                   // per-leaf tombstone bit mask (bit p = slot p is a tombstone),
                                   // then the guards per leaf

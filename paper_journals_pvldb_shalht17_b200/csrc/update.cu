@@ -695,8 +695,12 @@ __global__ void k_gflags(const uint64_t *__restrict__ tk, uint64_t n, uint32_t *
 // over the batch and two launches more).  status[0] is the tile counter, status[1 + t] tile t's
 // (flag:2 | count) word; the caller zeroes both.
 constexpr int GS_T = 1024, GS_I = 16, GS_TILE = GS_T * GS_I;   // 16K-item tiles: fewer look-back rounds
-__global__ void __launch_bounds__(GS_T) k_group_starts(const uint64_t *__restrict__ tk, uint64_t n,
+// (generic: items tk[i] >> shift of type K; hf / widx optional per-item outputs -- the head flag
+// and the exclusive head count, as UniqueSegments' flags + scan; widx[n] = the group count)
+template <typename K>
+__global__ void __launch_bounds__(GS_T) k_group_starts(const K *__restrict__ tk, uint64_t n, uint32_t shift,
                                                        uint32_t *__restrict__ gstart, uint32_t *__restrict__ ng_out,
+                                                       uint32_t *__restrict__ hf, uint32_t *__restrict__ widx,
                                                        unsigned long long *status, const Ctrl *c) {
   __shared__ uint32_t s_tile, s_prefix;
   __shared__ uint32_t wcnt[GS_T / 32];
@@ -713,9 +717,9 @@ __global__ void __launch_bounds__(GS_T) k_group_starts(const uint64_t *__restric
 #pragma unroll
   for (int j = 0; j < GS_I; ++j) {
     const uint64_t i = base + j * 32 + lane;
-    a[j] = i < n ? tk[i] : 0ull;
+    a[j] = i < n ? (uint64_t)(tk[i] >> shift) : 0ull;
   }
-  const uint64_t before = (lane == 0 && base > 0 && base <= n) ? tk[base - 1] : 0ull;
+  const uint64_t before = (lane == 0 && base > 0 && base <= n) ? (uint64_t)(tk[base - 1] >> shift) : 0ull;
   uint32_t bal[GS_I];
   uint32_t mine = 0;
   uint64_t carry = __shfl_sync(0xffffffffu, before, 0);
@@ -768,7 +772,8 @@ __global__ void __launch_bounds__(GS_T) k_group_starts(const uint64_t *__restric
       s_prefix = (uint32_t)prefix;
       if ((uint64_t)(tile + 1) * GS_TILE >= n) {        // last tile: the end sentinel and the count
         gstart[prefix + agg] = (uint32_t)n;
-        *ng_out = (uint32_t)(prefix + agg);
+        if (ng_out) *ng_out = (uint32_t)(prefix + agg);
+        if (widx) widx[n] = (uint32_t)(prefix + agg);
       }
     }
   }
@@ -777,9 +782,23 @@ __global__ void __launch_bounds__(GS_T) k_group_starts(const uint64_t *__restric
   const uint32_t lt = (1u << lane) - 1u;
 #pragma unroll
   for (int j = 0; j < GS_I; ++j) {
-    if ((bal[j] >> lane) & 1u) gstart[r + __popc(bal[j] & lt)] = (uint32_t)(base + j * 32 + lane);
+    const uint64_t i = base + j * 32 + lane;
+    const uint32_t f = (bal[j] >> lane) & 1u;
+    const uint32_t x = r + __popc(bal[j] & lt);
+    if (f) gstart[x] = (uint32_t)i;
+    if (widx && i < n) {
+      widx[i] = x;
+      hf[i] = f;
+    }
     r += __popc(bal[j]);
   }
+}
+
+// GPMA_GSTART_FUSED=0: group starts (level 0) and the segments of every
+// host-driven level by flags + scan + scatter (read per call)
+static bool gstart_fused() {
+  const char *e = getenv("GPMA_GSTART_FUSED");
+  return !e || atoi(e) != 0;
 }
 
 static gpma_status group_starts(gpma *g, const uint64_t *tk, uint64_t n, uint32_t *gstart, uint32_t *ng_out,
@@ -788,8 +807,8 @@ static gpma_status group_starts(gpma *g, const uint64_t *tk, uint64_t n, uint32_
   DevBuf &sb = tl_scan ? *tl_scan : g->b_scan;
   GP_CHECK(g, ensure(g, sb, (nt + 1) * sizeof(unsigned long long), s));
   GP_CHECK(g, fill_zero(g, sb.p, (nt + 1) * sizeof(unsigned long long), s));
-  GP_LAUNCH(g, k_group_starts, (unsigned)nt, GS_T, 0, s, tk, n, gstart, ng_out, (unsigned long long *)sb.p,
-            g->ctrl_d);
+  GP_LAUNCH(g, k_group_starts<uint64_t>, (unsigned)nt, GS_T, 0, s, tk, n, 0u, gstart, ng_out, (uint32_t *)nullptr,
+            (uint32_t *)nullptr, (unsigned long long *)sb.p, g->ctrl_d);
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
 }
@@ -2162,40 +2181,50 @@ __global__ void k_lvl_redistribute(Lvl a, uint64_t *__restrict__ key, uint32_t *
                                    uint32_t *__restrict__ cnt, uint32_t *__restrict__ tmask,
                                    uint64_t *__restrict__ row_offset, uint64_t bound,
                                    uint2 *__restrict__ dirty, uint64_t dirty_base) {
+  // 4 consecutive slots of one leaf per thread (L >= 4), stored as 16-B vectors; leaf bounds by
+  // shifts (Lc = 2^lvl leaves per window)
   const uint32_t nacc = a.aidx[a.p];
-  const uint64_t Lc = 1ull << a.lvl;
   const uint64_t wslots = (uint64_t)a.L << a.lvl;
-  const uint32_t lgw = (uint32_t)(__ffs(a.L) - 1) + a.lvl;        // wslots is a power of two
-  const uint64_t lim = min(bound, (uint64_t)nacc << lgw);         // the accepted windows' slots only
-  for (uint64_t g = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g < lim;
-       g += (uint64_t)gridDim.x * blockDim.x) {
-    uint64_t ai = g >> lgw;
+  const uint32_t lgL = (uint32_t)(__ffs(a.L) - 1);
+  const uint32_t lgw = lgL + a.lvl;                              // wslots is a power of two
+  const uint64_t lim = min(bound, (uint64_t)nacc << lgw) / 4;    // the accepted windows' slots only
+  for (uint64_t g4 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; g4 < lim;
+       g4 += (uint64_t)gridDim.x * blockDim.x) {
+    const uint64_t g = g4 * 4;
+    const uint64_t ai = g >> lgw;
     if (ai >= nacc) continue;
-    uint32_t w = a.alist[ai];
-    uint64_t N = a.nw[w];
-    uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
-    uint64_t off = g & (wslots - 1);
-    uint64_t l = leaf_div(off, a.L), p = leaf_mod(off, a.L);
-    uint64_t lo = l * N / Lc, hi = (l + 1) * N / Lc;
-    uint64_t s = leaf0 * a.L + off;
-    if (p < hi - lo) {
-      uint64_t e = a.woff[w] + lo + p;
-      uint64_t k = a.wk[e];
-      key[s] = k;
-      val[s] = a.wv[e];
-      if (is_guard_key(k)) row_offset[(k >> 32) - a.rb + 1] = s;
-    } else {
-      key[s] = KEY_NONE;
-      val[s] = 0;
+    const uint32_t w = a.alist[ai];
+    const uint64_t N = a.nw[w];
+    const uint64_t leaf0 = ((uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)) << a.lvl;
+    const uint64_t off = g & (wslots - 1);
+    const uint64_t l = off >> lgL, p = off & (a.L - 1);
+    const uint64_t lo = (l * N) >> a.lvl, hi = ((l + 1) * N) >> a.lvl, m = hi - lo;
+    const uint64_t s = leaf0 * a.L + off;
+    const uint64_t e0 = a.woff[w] + lo + p;
+    uint64_t k[4];
+    uint32_t v[4];
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      if (p + q < m) {
+        k[q] = a.wk[e0 + q];
+        v[q] = a.wv[e0 + q];
+        if (is_guard_key(k[q])) row_offset[(k[q] >> 32) - a.rb + 1] = s + q;
+      } else {
+        k[q] = KEY_NONE;
+        v[q] = 0;
+      }
     }
+    *reinterpret_cast<ulonglong2 *>(key + s) = make_ulonglong2(k[0], k[1]);
+    *reinterpret_cast<ulonglong2 *>(key + s + 2) = make_ulonglong2(k[2], k[3]);
+    *reinterpret_cast<uint4 *>(val + s) = make_uint4(v[0], v[1], v[2], v[3]);
     if (p == 0) {
-      cnt[leaf0 + l] = (uint32_t)(hi - lo);
+      cnt[leaf0 + l] = (uint32_t)m;
       tmask[leaf0 + l] = 0u;                          // tombstones are dropped by a rewrite
       uint32_t gc = 0;
       for (uint64_t e = lo; e < hi; ++e) gc += is_guard_key(a.wk[a.woff[w] + e]);
       tmask[a.nleaves + leaf0 + l] = gc;              // guards per leaf (third section)
     }
-    if (off == 0) dirty[dirty_base + ai] = make_uint2((uint32_t)leaf0, (uint32_t)Lc);
+    if (off == 0) dirty[dirty_base + ai] = make_uint2((uint32_t)leaf0, (uint32_t)(1ull << a.lvl));
   }
 }
 
@@ -2969,6 +2998,22 @@ __global__ void k_heads_all(const uint64_t *__restrict__ key, uint64_t *__restri
 }
 
 // Fix the heads of rewritten windows and of the run of empty leaves left of them.
+// Windows of >= HD_BIG leaves (levels >= 11 at L = 16, the root): a warp per window left a
+// 2^24-leaf root rewrite to one warp -- 350 ms for one configs[3] strict-delete batch -- so those
+// are fixed up by k_heads_span, a CTA per HD_BIG-leaf chunk of each big window.
+constexpr uint32_t HD_BIG = 2048;
+__global__ void k_heads_span(const uint64_t *__restrict__ key, uint64_t *__restrict__ head, uint32_t L,
+                             uint64_t nleaves, const uint2 *__restrict__ dirty) {
+  const uint2 wd = dirty[blockIdx.y];
+  const uint64_t l0 = (uint64_t)wd.x + (uint64_t)blockIdx.x * HD_BIG;
+  const uint64_t l1 = min(l0 + HD_BIG, (uint64_t)wd.x + wd.y);
+  for (uint64_t l = l0 + threadIdx.x; l < l1; l += blockDim.x) head[l] = next_head(key, L, nleaves, l);
+  if (blockIdx.x == 0 && threadIdx.x == 0) {             // empty leaves to the left carry the head
+    uint64_t hv = next_head(key, L, nleaves, wd.x);
+    for (int64_t m = (int64_t)wd.x - 1; m >= 0 && key[(uint64_t)m * L] == KEY_NONE; --m) head[m] = hv;
+  }
+}
+
 __global__ void k_heads_dirty(const uint64_t *__restrict__ key, uint64_t *__restrict__ head,
                               uint32_t L, uint64_t nleaves, const uint2 *__restrict__ dirty,
                               uint64_t ndirty) {
@@ -2976,6 +3021,7 @@ __global__ void k_heads_dirty(const uint64_t *__restrict__ key, uint64_t *__rest
   const uint64_t warps = (uint64_t)gridDim.x * (blockDim.x / 32);
   for (uint64_t d = (blockIdx.x * (uint64_t)blockDim.x + threadIdx.x) / 32; d < ndirty; d += warps) {
     uint2 wd = dirty[d];
+    if (wd.y >= HD_BIG) continue;                        // (k_heads_span: every SM on a big window)
     for (uint64_t l = wd.x + lane; l < (uint64_t)wd.x + wd.y; l += 32)
       head[l] = next_head(key, L, nleaves, l);
     if (lane == 0) {
@@ -3355,6 +3401,23 @@ static bool gather_big_on() {
   return !e || atoi(e) != 0;
 }
 
+// head fix-up of the windows rewritten by a batch's level loop: a warp per small window, a CTA
+// per HD_BIG-leaf chunk of every big one (recorded by level_step in g->big_dirty)
+static gpma_status fix_heads(gpma *g, uint64_t ndirty, cudaStream_t s) {
+  const uint64_t nl = g->cap / g->L;
+  const uint2 *dirty = (const uint2 *)g->b_dirty.p;
+  GP_LAUNCH(g, k_heads_dirty, grid_for(ndirty * 32), TB, 0, s, g->key, g->head, g->L, nl, dirty, ndirty);
+  for (const auto &b : g->big_dirty)
+    for (uint64_t y0 = 0; y0 < b[1]; y0 += 65535) {
+      const unsigned ny = (unsigned)std::min<uint64_t>(65535, b[1] - y0);
+      GP_LAUNCH(g, k_heads_span, dim3((unsigned)(b[2] / HD_BIG), ny), TB, 0, s, g->key, g->head, g->L, nl,
+                dirty + b[0] + y0);
+    }
+  g->big_dirty.clear();
+  GP_CHECK(g, cudaGetLastError());
+  return GPMA_OK;
+}
+
 static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t *dirty_base,
                               cudaStream_t s, bool resize_target, uint64_t new_cap, uint64_t *nk,
                               uint32_t *nv, uint32_t *ncnt, uint64_t *nhead = nullptr) {
@@ -3367,9 +3430,18 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
   if (small) {
     GP_LAUNCH(g, k_lvl_front_small, 1, LS_T, 0, s, a, g->cnt);
   } else {
-  GP_LAUNCH(g, k_lvl_flags, gp, TB, 0, s, a);
-  GP_CHECK(g, scan_u32(g, a.hf, a.widx, p, s));
-  GP_LAUNCH(g, k_lvl_first, gp, TB, 0, s, a);
+  if (gstart_fused()) {                                  // UniqueSegments (l.18-21) in one pass
+    const uint64_t nt = std::max<uint64_t>(1, (p + GS_TILE - 1) / GS_TILE);
+    DevBuf &sb = tl_scan ? *tl_scan : g->b_scan;
+    GP_CHECK(g, ensure(g, sb, (nt + 1) * sizeof(unsigned long long), s));
+    GP_CHECK(g, fill_zero(g, sb.p, (nt + 1) * sizeof(unsigned long long), s));
+    GP_LAUNCH(g, k_group_starts<uint32_t>, (unsigned)nt, GS_T, 0, s, a.pt, p, a.lvl, a.wfirst, (uint32_t *)nullptr,
+              a.hf, a.widx, (unsigned long long *)sb.p, g->ctrl_d);
+  } else {
+    GP_LAUNCH(g, k_lvl_flags, gp, TB, 0, s, a);
+    GP_CHECK(g, scan_u32(g, a.hf, a.widx, p, s));
+    GP_LAUNCH(g, k_lvl_first, gp, TB, 0, s, a);
+  }
   if (a.lvl <= 4) GP_LAUNCH(g, k_lvl_count<1>, grid_for(p), TB, 0, s, a, g->cnt);
   else if (a.lvl <= 11) GP_LAUNCH(g, k_lvl_count<32>, grid_for(p * 32), TB, 0, s, a, g->cnt);
   else {
@@ -3430,7 +3502,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     }
     if (a.op == GPMA_INSERT) GP_LAUNCH(g, k_lvl_place, gp, TB, 0, s, a, g->key, g->val);
     if (!resize_target) {
-      GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots), TB, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
+      GP_LAUNCH(g, k_lvl_redistribute, grid_for(bslots / 4), TB, 0, s, a, g->key, g->val, g->cnt, tmask_of(g),
                 g->row_offset, bslots, (uint2 *)g->b_dirty.p, *dirty_base);
     } else {
       // the single root window, laid out over the whole new array
@@ -3473,6 +3545,8 @@ merged:
   out->q = g->ctrl_h->sum & 0xFFFFFFFFull;
   out->nacc = g->ctrl_h->sum >> 32;
   out->p_new = g->ctrl_h->sum2;
+  if (out->nacc && ((uint64_t)1 << a.lvl) >= HD_BIG && !resize_target)
+    g->big_dirty.push_back({*dirty_base, out->nacc, (uint64_t)1 << a.lvl});
   *dirty_base += out->nacc;
   // compact the pending list into the other buffer
   if (out->p_new && !resize_target) {
@@ -3929,8 +4003,7 @@ static gpma_status gpma_lock_insert(gpma *g, uint64_t p, cudaStream_t s) {
       g->last.last_top_level = g->h + 1;
       if ((st = double_root(g, s))) return st;
     } else if (dirty_base) {
-      GP_LAUNCH(g, k_heads_dirty, grid_for(dirty_base * 32), TB, 0, s, g->key, g->head, g->L, nl,
-                (const uint2 *)g->b_dirty.p, dirty_base);
+      if ((st = fix_heads(g, dirty_base, s))) return st;
     }
     if (na) {                                           // the aborted insertions, sorted again
       Sorted srt;
@@ -4006,12 +4079,6 @@ static float interp_fv(gpma *g) {
   const char *e = getenv("GPMA_INTERP");
   if (e && atoi(e) == 0) return 0.f;
   return 1.0f / (float)std::max<uint32_t>(g->V, 1u);
-}
-
-// GPMA_GSTART_FUSED=0: group starts by flags + scan + scatter (read per call)
-static bool gstart_fused() {
-  const char *e = getenv("GPMA_GSTART_FUSED");
-  return !e || atoi(e) != 0;
 }
 
 static gpma_status upd_prefix(gpma *g, uint64_t *ik, uint32_t *iv, uint64_t n, int op, Sorted *srt,
@@ -4561,11 +4628,11 @@ static gpma_status first_accept_level(gpma *g, int cur, uint64_t p, uint32_t lvl
 static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int path,
                                        const Sorted &srt, cudaStream_t s) {
   gpma_status st;
-  const uint64_t nl = g->cap / g->L;
   uint32_t *keep2 = (uint32_t *)g->b_keep2.p, *kpos = (uint32_t *)g->b_kpos.p;
   const bool lock = op == GPMA_INSERT && g->algorithm == 1;   // GPMA (Alg. 1) instead of GPMA+
   const bool fused = !g->trace_on && !lock;
   if ((st = status_of(g))) return st;
+  g->big_dirty.clear();
   uint64_t p = (uint32_t)g->ctrl_h->sum;
   g->last.last_unique = g->ctrl_h->nunique;
   g->last.last_pending = p;
@@ -4704,8 +4771,7 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
     return resize(g, cur, p, op, s, &dirty_base);
   }
   if (dirty_base) {
-    GP_LAUNCH(g, k_heads_dirty, grid_for(dirty_base * 32), TB, 0, s, g->key, g->head, g->L, nl,
-              (const uint2 *)g->b_dirty.p, dirty_base);
+    if ((st = fix_heads(g, dirty_base, s))) return st;
   }
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;
