@@ -121,6 +121,8 @@ typedef struct {
   uint64_t last_pending_level1;    /* updates the leaves rejected (climbing to level 1)   */
   uint64_t last_levels_skipped;    /* levels a root-bound climb passed over (no window there
                                       could accept: dead-level skip)           */
+  uint64_t last_big_head_windows;  /* rewritten windows of >= 2048 leaves whose locate heads
+                                      were fixed up CTA-parallel              */
 } gpma_stats_t;
 
 /* Fill *cfg with the defaults above. */

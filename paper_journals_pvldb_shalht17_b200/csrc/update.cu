@@ -3407,12 +3407,14 @@ static gpma_status fix_heads(gpma *g, uint64_t ndirty, cudaStream_t s) {
   const uint64_t nl = g->cap / g->L;
   const uint2 *dirty = (const uint2 *)g->b_dirty.p;
   GP_LAUNCH(g, k_heads_dirty, grid_for(ndirty * 32), TB, 0, s, g->key, g->head, g->L, nl, dirty, ndirty);
-  for (const auto &b : g->big_dirty)
+  for (const auto &b : g->big_dirty) {
+    g->last.last_big_head_windows += b[1];
     for (uint64_t y0 = 0; y0 < b[1]; y0 += 65535) {
       const unsigned ny = (unsigned)std::min<uint64_t>(65535, b[1] - y0);
       GP_LAUNCH(g, k_heads_span, dim3((unsigned)(b[2] / HD_BIG), ny), TB, 0, s, g->key, g->head, g->L, nl,
                 dirty + b[0] + y0);
     }
+  }
   g->big_dirty.clear();
   GP_CHECK(g, cudaGetLastError());
   return GPMA_OK;

@@ -69,7 +69,8 @@ class gpma_stats_t(C.Structure):
                 ("last_resized", C.c_uint32), ("last_rounds", C.c_uint64), ("last_level0_windows", C.c_uint64),
                 ("total_batches", C.c_uint64), ("total_insert_keys", C.c_uint64), ("total_delete_keys", C.c_uint64),
                 ("total_slots_rewritten", C.c_uint64), ("total_windows_rewritten", C.c_uint64),
-                ("last_pending_level1", C.c_uint64), ("last_levels_skipped", C.c_uint64)]
+                ("last_pending_level1", C.c_uint64), ("last_levels_skipped", C.c_uint64),
+                ("last_big_head_windows", C.c_uint64)]
 
 
 _lib = None

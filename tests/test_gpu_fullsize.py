@@ -90,6 +90,7 @@ def test_config3_resize_stress_scaled():
     o = O.Oracle(V, pool[:live0].cpu(), vals[:live0].cpu(), delete_mode=O.REBALANCE)
     lo, hi = 0, live0          # live = pool[lo:hi]
     caps = [o.capacity]
+    big_heads = 0
     for step in range(146):
         if step < 70:
             ni, nd = 1 << 12, 1 << 10
@@ -102,6 +103,7 @@ def test_config3_resize_stress_scaled():
         o.insert(ik.cpu(), iv.cpu())
         g.delete(dk.contiguous())
         o.delete(dk.cpu())
+        big_heads += g.gpma_stats_host()["last_big_head_windows"]
         hi += ni
         lo += nd
         assert_same_layout(g, o, what=f"config3-scaled step {step}")
@@ -110,6 +112,7 @@ def test_config3_resize_stress_scaled():
     assert caps[-1] < max(caps), "no halving happened"
     assert g.gpma_stats()["resizes"] == o.stats()["resizes"]
     assert_same_csr(g, o, what="config3-scaled")
+    assert big_heads > 0, "no rewritten window of >= 2048 leaves (k_heads_span) was exercised"
 
 
 def _resize_pair(V, cap0, E0, seed, mode):
