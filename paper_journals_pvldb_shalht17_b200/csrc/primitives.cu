@@ -147,10 +147,10 @@ void pool_detach(gpma *g) {
 }
 
 // GPMA_TRACE_ALLOC=1: every allocation >= 64 MiB with its host time on stderr (diagnostics)
-static bool trace_alloc() {
-  static const bool on = [] {
+static int trace_alloc() {                              // 1: blocks >= 64 MiB, 2: >= 1 MiB
+  static const int on = [] {
     const char *e = getenv("GPMA_TRACE_ALLOC");
-    return e && atoi(e) != 0;
+    return e ? atoi(e) : 0;
   }();
   return on;
 }
@@ -200,7 +200,7 @@ cudaError_t dev_alloc(gpma *g, void **p, size_t bytes, cudaStream_t s) {
       }
     }
   }
-  if (trace_alloc() && bytes >= (64u << 20)) {
+  if (trace_alloc() && bytes >= (trace_alloc() > 1 ? (1u << 20) : (64u << 20))) {
     uint64_t res = 0, used = 0;
     if (!g->alloc_fn) {
       cudaMemPool_t pool = lib_pool(g->device);
