@@ -4589,6 +4589,73 @@ __global__ void k_lvl_first_accept(const uint32_t *__restrict__ pt, uint64_t p, 
   }
 }
 
+// Root reach (exact, the same invariant): an update reaches the root iff the test fails for every
+// window of its chain (levels lvl0 .. h-1); then the root is tested and re-lays out the whole
+// array -- in place or resized -- from all live entries and all pending updates, so every
+// rewrite of a lower window is overwritten and the levels below the root can be jumped over
+// (the layout is the same).  One thread per window of level lvl0 (its first pending update)
+// walks up its chain, the window bounds in the sorted pending list widened by exponential
+// searches, and stops at the first window that accepts (also its chain's absorption level:
+// the minimum over chains is the lowest accepting level, as k_lvl_first_accept).
+__device__ __forceinline__ uint64_t pend_lo(const uint32_t *pt, uint64_t lo, uint32_t l, uint32_t w) {
+  // pt[lo] is in window w (pt >> l is non-decreasing): the window's first index
+  uint64_t good = lo, step = 1, bad;
+  for (;;) {
+    if (good == 0) return 0;
+    const uint64_t probe = good > step ? good - step : 0;
+    if ((pt[probe] >> l) == w) {
+      good = probe;
+      step <<= 1;
+    } else {
+      bad = probe;
+      break;
+    }
+  }
+  while (bad + 1 < good) {                               // pt[bad] outside, pt[good] inside
+    const uint64_t mid = (bad + good) >> 1;
+    if ((pt[mid] >> l) == w) good = mid;
+    else bad = mid;
+  }
+  return good;
+}
+__device__ __forceinline__ uint64_t pend_hi(const uint32_t *pt, uint64_t p, uint64_t hi, uint32_t l, uint32_t w) {
+  uint64_t lo = hi, step = 1;                            // first index past the window
+  while (hi < p && (pt[hi] >> l) == w) {
+    lo = hi + 1;
+    hi += step;
+    step <<= 1;
+  }
+  if (hi > p) hi = p;
+  while (lo < hi) {
+    const uint64_t mid = (lo + hi) >> 1;
+    if ((pt[mid] >> l) == w) lo = mid + 1;
+    else hi = mid;
+  }
+  return lo;
+}
+__global__ void k_lvl_root_reach(const uint32_t *__restrict__ pt, uint64_t p, const uint32_t *__restrict__ pre,
+                                 uint32_t lvl0, uint32_t lvl1, LvlBound tb, int op, uint32_t *first,
+                                 uint32_t *root) {
+  for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < p; i += (uint64_t)gridDim.x * blockDim.x) {
+    const uint32_t t = pt[i];
+    if (i && (pt[i - 1] >> lvl0) == (t >> lvl0)) continue;   // not its level-lvl0 window's first
+    uint64_t lo = i, hi = i + 1;
+    bool passed = false;
+    for (uint32_t l = lvl0; l < lvl1 && !passed; ++l) {
+      const uint32_t w = t >> l;
+      lo = pend_lo(pt, lo, l, w);
+      hi = pend_hi(pt, p, hi, l, w);
+      const uint64_t n = (uint64_t)(pre[(uint64_t)(w + 1) << l] - pre[(uint64_t)w << l]);
+      const uint64_t u = hi - lo;
+      if (op == GPMA_INSERT ? n + u <= tb.t[l] : (n >= u && n - u >= tb.t[l])) {
+        atomicMin(first, l);
+        passed = true;
+      }
+    }
+    if (!passed) atomicOr(root, 1u);
+  }
+}
+
 // GPMA_TRACE_LEVELS=1: every host-driven level of a batch on stderr (diagnostics)
 static bool trace_levels() {
   static const bool on = [] {
@@ -4607,22 +4674,38 @@ constexpr uint64_t SKIP_MINP = 256;     // pending updates worth the prefix of t
 
 // the lowest level in [lvl0, lvl1) at which a window of the pending list (buffers cur) accepts,
 // lvl1 if none
+// (root != nullptr: the per-chain walk of k_lvl_root_reach, which also tells whether some update
+// reaches the root)
 static gpma_status first_accept_level(gpma *g, int cur, uint64_t p, uint32_t lvl0, uint32_t lvl1, int op,
-                                      uint32_t *out, cudaStream_t s) {
+                                      uint32_t *out, cudaStream_t s, bool *root = nullptr) {
   const uint64_t nl = g->cap / g->L;
-  GP_CHECK(g, ensure(g, g->b_misc3, (nl + 2) * 4, s));
-  uint32_t *pre = (uint32_t *)g->b_misc3.p, *first = pre + nl + 1;
+  GP_CHECK(g, ensure(g, g->b_misc3, (nl + 4) * 4, s));
+  uint32_t *pre = (uint32_t *)g->b_misc3.p, *first = pre + nl + 1, *rf = pre + nl + 2;
   GP_CHECK(g, scan_u32(g, g->cnt, pre, nl, s));
   GP_LAUNCH(g, k_set_u32, 1, 1, 0, s, first, lvl1);
+  if (root) GP_LAUNCH(g, k_set_u32, 1, 1, 0, s, rf, 0u);
   LvlBound tb{};
   const std::vector<uint64_t> &b = op == GPMA_INSERT ? g->tmax : g->tmin;
   for (uint32_t j = 0; j < 64 && j < b.size(); ++j) tb.t[j] = b[j];
-  GP_LAUNCH(g, k_lvl_first_accept, grid_for(p), TB, 0, s, (const uint32_t *)g->b_pt[cur].p, p, pre, lvl0, lvl1, tb,
-            op, first);
-  GP_CHECK(g, readback(g, g->pin, first, 4, s));
+  if (root)
+    GP_LAUNCH(g, k_lvl_root_reach, grid_for(p), TB, 0, s, (const uint32_t *)g->b_pt[cur].p, p, pre, lvl0, lvl1, tb,
+              op, first, rf);
+  else
+    GP_LAUNCH(g, k_lvl_first_accept, grid_for(p), TB, 0, s, (const uint32_t *)g->b_pt[cur].p, p, pre, lvl0, lvl1,
+              tb, op, first);
+  GP_CHECK(g, readback(g, g->pin, first, 8, s));
   GP_CHECK(g, cudaStreamSynchronize(s));
-  memcpy(out, g->pin, 4);
+  uint32_t w2[2];
+  memcpy(w2, g->pin, 8);
+  *out = w2[0];
+  if (root) *root = w2[1] != 0;
   return GPMA_OK;
+}
+
+// GPMA_ROOT_JUMP=0 disables the root-reach jump (read per call)
+static bool root_jump_on() {
+  const char *e = getenv("GPMA_ROOT_JUMP");
+  return !e || atoi(e) != 0;
 }
 
 // After the prefix's host round trip: the pending list of level 1 (if any), the level loop, the
@@ -4759,10 +4842,14 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
               std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - tl_call_start).count());
     if (skip && p >= SKIP_MINP && 2 * p > p_in && lvl + 1 < g->h && lvl >= next_check) {
       // a level that absorbed less than half of many pending updates: likely a root-bound climb
-      // -- jump over the levels where no window accepts (nothing happens there).  A check that
-      // finds the next level accepting backs off for two levels.
+      // -- jump over the levels where no window accepts (nothing happens there), or, when some
+      // update reaches the root (absorbed less than a fifth: the root-reach walk), straight to
+      // the root.  A check that finds the next level accepting backs off for two levels.
       uint32_t j = 0;
-      if ((st = first_accept_level(g, cur, p, lvl + 1, g->h, op, &j, s))) return st;
+      bool root = false;
+      const bool rj = root_jump_on() && 5 * (p_in - p) < p_in;
+      if ((st = first_accept_level(g, cur, p, lvl + 1, g->h, op, &j, s, rj ? &root : nullptr))) return st;
+      if (root) j = g->h;
       g->last.last_levels_skipped += j - (lvl + 1);
       if (j == lvl + 1) next_check = lvl + 3;
       lvl = j - 1;

@@ -274,8 +274,12 @@ def test_dead_level_skip_intermediate_and_root(mode):
         finally:
             os.environ.pop("GPMA_LVL_SKIP", None)
     (si1, sd1), (si0, sd0) = stats
-    keys = ("last_top_level", "last_windows_rewritten", "last_slots_rewritten", "capacity", "resizes")
-    assert {k: si1[k] for k in keys} == {k: si0[k] for k in keys}
-    assert {k: sd1[k] for k in keys} == {k: sd0[k] for k in keys}
+    # (windows / slots rewritten only where no update reaches the root: a root-reaching climb jumps
+    # to the root, whose rewrite supersedes the lower ones -- same layout, fewer rewrites)
+    def keys(st):
+        k = ("last_top_level", "capacity", "resizes")
+        return k + (("last_windows_rewritten", "last_slots_rewritten") if st["last_top_level"] < st["height"] else ())
+    assert {k: si1[k] for k in keys(si1)} == {k: si0[k] for k in keys(si1)}
+    assert {k: sd1[k] for k in keys(sd1)} == {k: sd0[k] for k in keys(sd1)}
     assert si1["last_levels_skipped"] > 0 and si0["last_levels_skipped"] == 0
     assert si1["last_top_level"] <= si1["height"], "the hot batch should be absorbed below the root"
