@@ -257,12 +257,14 @@ cudaError_t ensure(gpma *g, DevBuf &b, size_t bytes, cudaStream_t s) {
   if (bytes == 0) bytes = 16;
   if (b.bytes >= bytes) return cudaSuccess;
   size_t want = std::max(bytes, b.bytes + b.bytes / 2);
-  // Large scratch in power-of-two sizes: the pool serves a request from one free chunk, and
+  // Scratch >= 1 MiB in power-of-two sizes: the pool serves a request from one free chunk, and
   // chunks freed by a previous store / scratch of another size made it re-map fragmented free
   // memory (8-14 ms per 256-512 MiB request with the pool's reserved size unchanged,
-  // tools/resize_trace.py with GPMA_TRACE_ALLOC=1); equal size classes reuse whole chunks.
-  if (want >= (64u << 20)) {
-    size_t p2 = 64u << 20;
+  // tools/resize_trace.py with GPMA_TRACE_ALLOC=1; 1-5 ms, sometimes 40-80 ms, for the 14-32 MiB
+  // level buffers of the configs[3] grow phase, tools/step_trace.py); equal size classes reuse
+  // whole chunks.
+  if (want >= (1u << 20)) {
+    size_t p2 = 1u << 20;
     while (p2 < want) p2 <<= 1;
     want = p2;
   }
