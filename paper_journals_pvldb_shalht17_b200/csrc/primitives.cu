@@ -33,14 +33,14 @@ struct DevPool {
 };
 DevPool g_pools[64];
 
-// Blocks >= 64 MiB (store arrays, root-merge and level scratch) freed by the library are kept in a
+// Blocks >= 1 MiB (store arrays, root-merge and level scratch) freed by the library are kept in a
 // per-device cache keyed by exact size and handed back to the next request of that size, with
 // an event ordering the reuse after the freeing stream's work.  The pool alone re-mapped
 // fragmented free memory for such requests with its reserved size unchanged: 140-510 ms for
 // one 0.5-2 GiB request in a resizing step (tools/resize_trace.py, GPMA_TRACE_ALLOC=1).
 // GPMA_BLOCK_CACHE=0 disables it.  The cache is emptied into the pool when an allocation
 // fails (then the request is retried) and trimmed with the pool on the last destroy.
-constexpr size_t BIG_BLOCK = 64u << 20;
+constexpr size_t BIG_BLOCK = 1u << 20;
 struct CachedBlock {
   void *p;
   size_t bytes;
