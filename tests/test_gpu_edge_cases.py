@@ -110,7 +110,7 @@ def test_halving_down_to_minimum_capacity():
     assert st["capacity"] == o.capacity and st["live_edges"] == 0
 
 
-@pytest.mark.parametrize("n", [2047, 2048, 2049, 4095, 4096, 4097, 12289, 300_001])
+@pytest.mark.parametrize("n", [2047, 2048, 2049, 4095, 4096, 4097, 8191, 12288, 12289, 300_001])
 def test_sort_tiles_and_stability(n):
     """Batch sizes around the small-sort limit (2048) and the onesweep tile (4096 keys), with
     heavy duplication and distinct values: the stable sort must let the LAST copy of every key
