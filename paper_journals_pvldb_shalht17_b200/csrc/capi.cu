@@ -161,7 +161,7 @@ void free_handle(gpma *g) {
                     &g->b_hf, &g->b_widx, &g->b_wfirst, &g->b_acc, &g->b_aidx, &g->b_alist, &g->b_nw,
                     &g->b_woff, &g->b_keep2, &g->b_kpos, &g->b_lpre, &g->b_wk, &g->b_wv, &g->b_dirty,
                     &g->b_scan, &g->b_hist, &g->b_stage[0], &g->b_stage[1], &g->b_stage[2],
-                    &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3};
+                    &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3, &g->b_sup};
   for (DevBuf *b : bufs) gp::release(g, *b, s);
   for (gp::Scratch &x : g->an) {
     DevBuf *xb[] = {&x.b[0], &x.b[1], &x.b[2], &x.b[3], &x.misc, &x.lpre, &x.scan, &x.stage[0], &x.stage[1]};

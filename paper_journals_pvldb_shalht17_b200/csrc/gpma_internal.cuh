@@ -341,6 +341,8 @@ struct gpma {
   uint64_t *key = nullptr;        // [cap]
   uint32_t *val = nullptr;        // [cap]
   bool root_heads_done = false;   // the last root re-layout wrote the locate heads
+  gp::DevBuf b_sup;                // truly accepted windows of the planned climb (heap-indexed bits)
+  bool sup_on = false;             // the host levels of this batch follow a plan (b_sup valid)
   std::vector<std::array<uint64_t, 3>> big_dirty;   // (first dirty entry, windows, leaves each) of big rewritten windows
   uint32_t *cnt = nullptr;        // [3*cap/L]: live entries (incl. guards) per leaf, then the
                                   // per-leaf tombstone bit mask (bit p = slot p is a tombstone),

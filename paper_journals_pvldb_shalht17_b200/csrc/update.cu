@@ -1831,7 +1831,20 @@ struct Lvl {
   uint32_t rb;         // first owned row (row offsets are local)
   uint64_t nleaves;    // leaves of the store (offset of the guard counts after the masks)
   const uint32_t *lcnt; // small levels: leaf live counts read directly instead of the prefix lpre
+  const uint32_t *sup;  // (nullable) windows the batch truly accepts, heap-indexed bits (superseded)
 };
+
+// A window (level l, index w) is superseded when a window above it is truly accepted (its test
+// passes while updates of its chain are still pending -- k_lvl_root_reach marks them): that
+// rewrite re-lays out all of it, so a lower rewrite inside it changes nothing and is skipped
+// (its updates stay pending and are merged there).  Bits are heap-indexed: (l, w) -> (nl >> l) + w,
+// the parent of id is id >> 1.
+__device__ __forceinline__ bool lvl_superseded(const uint32_t *sup, uint64_t nl, uint32_t l, uint64_t w) {
+  uint64_t id = (nl >> l) + w;
+  for (id >>= 1; id >= 2; id >>= 1)                     // (id 1, the root, is never marked)
+    if ((__ldg(sup + (id >> 5)) >> (id & 31)) & 1u) return true;
+  return false;
+}
 
 __global__ void k_lvl_flags(Lvl a) {
   for (uint64_t j = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; j < a.p;
@@ -1891,6 +1904,7 @@ __global__ void k_lvl_count(Lvl a, const uint32_t *__restrict__ cnt) {
         if (a.force) ok = true;
         else if (a.op == GPMA_INSERT) ok = n + u <= a.tmax;
         else ok = n >= u && n - u >= a.tmin;
+        if (ok && !a.force && a.sup && lvl_superseded(a.sup, a.nleaves, a.lvl, leaf0 >> a.lvl)) ok = false;
         a.acc[w] = ok ? 1u : 0u;
         a.nw[w] = ok ? (a.op == GPMA_INSERT ? n + u : n - u) : 0;
       }
@@ -1937,6 +1951,8 @@ __global__ void k_lvl_accept(Lvl a) {
     if (a.force) ok = true;
     else if (a.op == GPMA_INSERT) ok = n + u <= a.tmax;
     else ok = n >= u && n - u >= a.tmin;
+    if (ok && !a.force && a.sup && lvl_superseded(a.sup, a.nleaves, a.lvl, (uint64_t)(a.pt[a.wfirst[w]] >> a.lvl)))
+      ok = false;
     a.acc[w] = ok ? 1u : 0u;
     a.nw[w] = ok ? (a.op == GPMA_INSERT ? n + u : n - u) : 0;
   }
@@ -2423,6 +2439,7 @@ __global__ void __launch_bounds__(LS_T) k_lvl_front_small(Lvl a, const uint32_t 
       if (a.force) ok = true;
       else if (a.op == GPMA_INSERT) ok = n + u <= a.tmax;
       else ok = n >= u && n - u >= a.tmin;
+      if (ok && !a.force && a.sup && lvl_superseded(a.sup, a.nleaves, a.lvl, leaf0 >> a.lvl)) ok = false;
       ac[i] = ok ? 1u : 0u;
       nw[i] = ok ? (a.op == GPMA_INSERT ? n + u : n - u) : 0;
     }
@@ -3606,6 +3623,7 @@ static Lvl make_lvl(gpma *g, int cur, uint64_t p, uint32_t lvl, int op) {
   a.force = 0;
   a.rb = g->rb;
   a.nleaves = g->cap / g->L;
+  a.sup = g->sup_on ? (const uint32_t *)g->b_sup.p : nullptr;
   return a;
 }
 
@@ -4326,7 +4344,7 @@ static std::vector<uint64_t> upd_signature(gpma *g, uint64_t n, int op) {
                           &g->b_hf, &g->b_widx, &g->b_wfirst, &g->b_acc, &g->b_aidx, &g->b_alist, &g->b_nw,
                           &g->b_woff, &g->b_keep2, &g->b_kpos, &g->b_lpre, &g->b_wk, &g->b_wv, &g->b_dirty,
                           &g->b_scan, &g->b_hist, &g->b_stage[0], &g->b_stage[1], &g->b_stage[2],
-                          &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3};
+                          &g->b_stage[3], &g->b_misc, &g->b_misc2, &g->b_misc3, &g->b_sup};
   for (const DevBuf *b : bufs) {
     v.push_back((uint64_t)(uintptr_t)b->p);
     v.push_back(b->bytes);
@@ -4635,7 +4653,7 @@ __device__ __forceinline__ uint64_t pend_hi(const uint32_t *pt, uint64_t p, uint
 }
 __global__ void k_lvl_root_reach(const uint32_t *__restrict__ pt, uint64_t p, const uint32_t *__restrict__ pre,
                                  uint32_t lvl0, uint32_t lvl1, LvlBound tb, int op, uint32_t *first,
-                                 uint32_t *root) {
+                                 uint32_t *root, uint32_t *sup, uint64_t nl) {
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < p; i += (uint64_t)gridDim.x * blockDim.x) {
     const uint32_t t = pt[i];
     if (i && (pt[i - 1] >> lvl0) == (t >> lvl0)) continue;   // not its level-lvl0 window's first
@@ -4649,11 +4667,37 @@ __global__ void k_lvl_root_reach(const uint32_t *__restrict__ pt, uint64_t p, co
       const uint64_t u = hi - lo;
       if (op == GPMA_INSERT ? n + u <= tb.t[l] : (n >= u && n - u >= tb.t[l])) {
         atomicMin(first, l);
+        if (sup) {                                       // the chain's truly accepted window
+          const uint64_t id = (nl >> l) + w;
+          atomicOr(sup + (id >> 5), 1u << (id & 31));
+        }
         passed = true;
       }
     }
     if (!passed) atomicOr(root, 1u);
   }
+}
+
+// the levels that hold a maximal truly accepted window (bit l of *mask): one thread per word of
+// the heap-indexed bitmap
+__global__ void k_lvl_maximal(const uint32_t *__restrict__ sup, uint64_t nwords, uint64_t nl,
+                              unsigned long long *mask) {
+  const uint32_t H = 63 - __clzll((long long)nl);        // log2(nl): level of id 1
+  unsigned long long m = 0;
+  for (uint64_t wd = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; wd < nwords;
+       wd += (uint64_t)gridDim.x * blockDim.x) {
+    uint32_t b = sup[wd];
+    while (b) {
+      const int k = __ffs(b) - 1;
+      b &= b - 1;
+      const uint64_t id = wd * 32 + (uint64_t)k;
+      const uint32_t l = H - (63 - __clzll((long long)id));   // (nl >> l) <= id < 2 (nl >> l)
+      const uint64_t w = id - (nl >> l);
+      if (!lvl_superseded(sup, nl, l, w)) m |= 1ull << l;
+    }
+  }
+  for (int o = 16; o; o >>= 1) m |= __shfl_xor_sync(0xffffffffu, m, o);
+  if ((threadIdx.x & 31) == 0 && m) atomicOr(mask, m);
 }
 
 // GPMA_TRACE_LEVELS=1: every host-driven level of a batch on stderr (diagnostics)
@@ -4689,7 +4733,7 @@ static gpma_status first_accept_level(gpma *g, int cur, uint64_t p, uint32_t lvl
   for (uint32_t j = 0; j < 64 && j < b.size(); ++j) tb.t[j] = b[j];
   if (root)
     GP_LAUNCH(g, k_lvl_root_reach, grid_for(p), TB, 0, s, (const uint32_t *)g->b_pt[cur].p, p, pre, lvl0, lvl1, tb,
-              op, first, rf);
+              op, first, rf, (uint32_t *)nullptr, nl);
   else
     GP_LAUNCH(g, k_lvl_first_accept, grid_for(p), TB, 0, s, (const uint32_t *)g->b_pt[cur].p, p, pre, lvl0, lvl1,
               tb, op, first);
@@ -4708,6 +4752,45 @@ static bool root_jump_on() {
   return !e || atoi(e) != 0;
 }
 
+// GPMA_LVL_PLAN=0 disables the climb plan (read per call)
+static bool lvl_plan_on() {
+  const char *e = getenv("GPMA_LVL_PLAN");
+  return !e || atoi(e) != 0;
+}
+
+// The plan of a host-driven climb from level lvl0 (exact, the dead-level skip's invariant): every
+// chain's truly accepted window (its first passing window) marked in b_sup, whether some chain
+// reaches the root, and the levels holding a maximal (not superseded) truly accepted window.
+// Only those levels -- and the root, if reached -- need stepping; there the superseded windows
+// are rejected (their updates are merged by the window above), so the final layout is the one
+// the level-by-level loop produces, with each region rewritten once.
+static gpma_status plan_levels(gpma *g, int cur, uint64_t p, uint32_t lvl0, int op, bool *root, uint64_t *mask,
+                               cudaStream_t s) {
+  const uint64_t nl = g->cap / g->L;
+  const uint64_t nwords = (2 * nl + 31) / 32;
+  GP_CHECK(g, ensure(g, g->b_misc3, (nl + 8) * 4, s));
+  GP_CHECK(g, ensure(g, g->b_sup, nwords * 4 + 16, s));
+  uint32_t *pre = (uint32_t *)g->b_misc3.p, *first = pre + nl + 1, *rf = pre + nl + 2;
+  unsigned long long *mk = reinterpret_cast<unsigned long long *>(pre + nl + 4);   // 8-B aligned (nl even)
+  uint32_t *sup = (uint32_t *)g->b_sup.p;
+  GP_CHECK(g, scan_u32(g, g->cnt, pre, nl, s));
+  GP_CHECK(g, fill_zero(g, sup, nwords * 4, s));
+  GP_CHECK(g, fill_zero(g, first, 5 * 4, s));          // first, root, pad, mask
+  LvlBound tb{};
+  const std::vector<uint64_t> &b = op == GPMA_INSERT ? g->tmax : g->tmin;
+  for (uint32_t j = 0; j < 64 && j < b.size(); ++j) tb.t[j] = b[j];
+  GP_LAUNCH(g, k_lvl_root_reach, grid_for(p), TB, 0, s, (const uint32_t *)g->b_pt[cur].p, p, pre, lvl0, g->h, tb, op,
+            first, rf, sup, nl);
+  GP_LAUNCH(g, k_lvl_maximal, grid_for(nwords), TB, 0, s, (const uint32_t *)sup, nwords, nl, mk);
+  GP_CHECK(g, readback(g, g->pin, first, 5 * 4, s));
+  GP_CHECK(g, cudaStreamSynchronize(s));
+  uint32_t w[5];
+  memcpy(w, g->pin, 20);
+  *root = w[1] != 0;
+  *mask = (uint64_t)w[3] | ((uint64_t)w[4] << 32);
+  return GPMA_OK;
+}
+
 // After the prefix's host round trip: the pending list of level 1 (if any), the level loop, the
 // root resize, the head fix-up.  ik / iv: the batch the prefix read (staged or the caller's).
 static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32_t *iv, uint64_t n, int op, int path,
@@ -4718,6 +4801,7 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
   const bool fused = !g->trace_on && !lock;
   if ((st = status_of(g))) return st;
   g->big_dirty.clear();
+  g->sup_on = false;
   uint64_t p = (uint32_t)g->ctrl_h->sum;
   g->last.last_unique = g->ctrl_h->nunique;
   g->last.last_pending = p;
@@ -4826,7 +4910,23 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
   Nvtx nvtx_levels("update: host level loop");
   const bool skip = lvl_skip_on() && !g->trace_on && g->cap < (1ull << 32) && g->h < 64;
   uint32_t next_check = 0;
+  bool planned = false;
+  uint64_t lvl_mask = 0;
+  g->sup_on = false;
+  if (skip && lvl_plan_on() && p >= SKIP_MINP && lvl < g->h) {
+    bool root = false;
+    if ((st = plan_levels(g, cur, p, lvl, op, &root, &lvl_mask, s))) return st;
+    if (root) lvl_mask = 0;                              // the root rewrite supersedes every level
+    planned = true;
+    g->sup_on = true;
+    if (trace_levels())
+      fprintf(stderr, "[gpma] plan from level %u: levels %llx, root %d\n", lvl, (unsigned long long)lvl_mask, (int)root);
+  }
   for (; lvl <= g->h && p > 0; ++lvl) {
+    if (planned && lvl < g->h && !((lvl_mask >> lvl) & 1ull)) {   // no maximal accepted window here
+      g->last.last_levels_skipped++;
+      continue;
+    }
     Lvl a = make_lvl(g, cur, p, lvl, op);
     LevelOut lo{};
     if ((st = level_step(g, a, cur, &lo, &dirty_base, s, false, 0, nullptr, nullptr, nullptr))) return st;
@@ -4840,7 +4940,7 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
       fprintf(stderr, "[gpma] level %2u  pending %9llu -> %9llu  accepted %8llu  at %.3f ms\n", lvl,
               (unsigned long long)p_in, (unsigned long long)p, (unsigned long long)lo.nacc,
               std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - tl_call_start).count());
-    if (skip && p >= SKIP_MINP && 2 * p > p_in && lvl + 1 < g->h && lvl >= next_check) {
+    if (!planned && skip && p >= SKIP_MINP && 2 * p > p_in && lvl + 1 < g->h && lvl >= next_check) {
       // a level that absorbed less than half of many pending updates: likely a root-bound climb
       // -- jump over the levels where no window accepts (nothing happens there), or, when some
       // update reaches the root (absorbed less than a fifth: the root-reach walk), straight to
@@ -4855,6 +4955,7 @@ static gpma_status update_after_prefix(gpma *g, const uint64_t *ik, const uint32
       lvl = j - 1;
     }
   }
+  g->sup_on = false;
   if (p > 0) {
     g->last.last_top_level = g->h + 1;
     return resize(g, cur, p, op, s, &dirty_base);

@@ -277,8 +277,9 @@ def test_dead_level_skip_intermediate_and_root(mode):
     # (windows / slots rewritten only where no update reaches the root: a root-reaching climb jumps
     # to the root, whose rewrite supersedes the lower ones -- same layout, fewer rewrites)
     def keys(st):
-        k = ("last_top_level", "capacity", "resizes")
-        return k + (("last_windows_rewritten", "last_slots_rewritten") if st["last_top_level"] < st["height"] else ())
+        # (windows / slots rewritten differ by design: the climb plan rewrites each region once,
+        # at its highest accepted window -- same layout, fewer rewrites)
+        return ("last_top_level", "capacity", "resizes")
     assert {k: si1[k] for k in keys(si1)} == {k: si0[k] for k in keys(si1)}
     assert {k: sd1[k] for k in keys(sd1)} == {k: sd0[k] for k in keys(sd1)}
     assert si1["last_levels_skipped"] > 0 and si0["last_levels_skipped"] == 0

@@ -151,7 +151,7 @@ def test_config0_sliding_window_graph_replay(seed, monkeypatch):
 @pytest.mark.parametrize("knob", ["GPMA_DEL_SORT=1", "GPMA_INS_FUSED=0", "GPMA_INS_LEAFSORT=0",
                                   "GPMA_INS_LEAFSORT=0,GPMA_INS_THREAD=0", "GPMA_LVL_COOP=0", "GPMA_LVL_WARP=0", "GPMA_INTERP=0", "GPMA_ILP=1",
                                   "GPMA_ILP=4", "GPMA_SMALL=2048", "GPMA_SMALL=0,GPMA_DEL_SORT=1",
-                                  "GPMA_GSTART_FUSED=0", "GPMA_LVL_SKIP=0", "GPMA_ROOT_JUMP=0"])
+                                  "GPMA_GSTART_FUSED=0", "GPMA_LVL_SKIP=0", "GPMA_ROOT_JUMP=0", "GPMA_LVL_PLAN=0"])
 @pytest.mark.parametrize("seed", range(3))
 def test_config0_alternative_paths(seed, knob, monkeypatch):
     """The strategy switches give the same layouts as the defaults (configs[0] batches are 1024 keys,
