@@ -2057,7 +2057,38 @@ __global__ void k_lvl_gather(Lvl a, const uint64_t *__restrict__ key, const uint
 // of a few shared-memory entries instead of ~log2(pending) dependent global probes (merge-path
 // split of the window merge, Alg. 4 l.26).
 constexpr int GB_T = 256, GB_I = 16, GB_CHUNK = GB_T * GB_I, GB_SP = 4096;
-__global__ void __launch_bounds__(GB_T) k_lvl_gather_big(Lvl a, const uint64_t *__restrict__ key,
+// CTAs per SM of the big-window gather (GPMA_GB_PER_SM; 4 / 8 / 16 measured alike)
+static int gb_per_sm() {
+  const char *e = getenv("GPMA_GB_PER_SM");
+  return e ? std::max(1, atoi(e)) : 8;
+}
+
+// first index in [lo, hi) with a[i] >= x (hi if none), all 32 lanes of a warp: 32 probes per
+// round narrow the range 32-fold (4 rounds for 10^6 keys instead of 20 dependent probes)
+__device__ __forceinline__ uint64_t warp_lower_bound_u64(const uint64_t *__restrict__ a, uint64_t lo, uint64_t hi,
+                                                         uint64_t x) {
+  const int lane = threadIdx.x & 31;
+  while (hi - lo > 32) {
+    const uint64_t step = (hi - lo + 31) / 32;
+    const uint64_t idx = lo + (uint64_t)lane * step;
+    const bool ge = idx >= hi || a[idx] >= x;            // (past the range counts as >= x)
+    const uint32_t m = __ballot_sync(0xffffffffu, ge);
+    if (m & 1u) return lo;                               // a[lo] >= x
+    if (m == 0) {                                        // every probe < x: past the last one
+      lo = lo + 31 * step + 1;
+    } else {
+      const int f = __ffs(m) - 1;                        // answer in (probe f-1, probe f]
+      const uint64_t pf = lo + (uint64_t)f * step;
+      lo = lo + (uint64_t)(f - 1) * step + 1;
+      hi = min(hi, pf);
+    }
+  }
+  const uint64_t idx = lo + lane;
+  const bool ge = idx >= hi || a[idx] >= x;
+  const uint32_t m = __ballot_sync(0xffffffffu, ge);
+  return m ? min(hi, lo + (uint64_t)(__ffs(m) - 1)) : hi;
+}
+__global__ void __launch_bounds__(GB_T, 4) k_lvl_gather_big(Lvl a, const uint64_t *__restrict__ key,
                                                           const uint32_t *__restrict__ val, uint64_t nchunks) {
   __shared__ uint64_t sp[GB_SP];
   __shared__ uint64_t red_min[GB_T / 32], red_max[GB_T / 32];
@@ -2101,7 +2132,7 @@ __global__ void __launch_bounds__(GB_T) k_lvl_gather_big(Lvl a, const uint64_t *
     }
     __syncthreads();
     const uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
-    if (threadIdx.x == 0) {
+    if (warp == 0) {                                     // the chunk's pending run: warp-wide searches
       uint64_t mn = KEY_NONE, mx = 0;
       for (int q = 0; q < GB_T / 32; ++q) {
         mn = min(mn, red_min[q]);
@@ -2109,11 +2140,13 @@ __global__ void __launch_bounds__(GB_T) k_lvl_gather_big(Lvl a, const uint64_t *
       }
       uint64_t pa = ub, pb = ub;
       if (mn != KEY_NONE) {
-        pa = lower_bound_u64(a.pk, ub, ue, mn);
-        pb = lower_bound_u64(a.pk, pa, ue, mx == KEY_NONE ? mx : mx + 1);
+        pa = warp_lower_bound_u64(a.pk, ub, ue, mn);
+        pb = mx == KEY_NONE ? ue : warp_lower_bound_u64(a.pk, pa, ue, mx + 1);
       }
-      s_pa = pa;
-      s_pb = pb;
+      if (lane == 0) {
+        s_pa = pa;
+        s_pb = pb;
+      }
     }
     __syncthreads();
     const uint64_t pa = s_pa, pb = s_pb;
@@ -3514,7 +3547,7 @@ static gpma_status level_step(gpma *g, Lvl &a, int cur, LevelOut *out, uint64_t 
     uint64_t bslots_r = (bslots + 31) & ~31ull;
     if (a.lvl && wslots >= (uint64_t)GB_CHUNK && gather_big_on()) {
       const uint64_t nch = bslots / GB_CHUNK;
-      GP_LAUNCH(g, k_lvl_gather_big, (unsigned)std::min<uint64_t>(nch, (uint64_t)num_sms() * 8), GB_T, 0, s, a, g->key,
+      GP_LAUNCH(g, k_lvl_gather_big, (unsigned)std::min<uint64_t>(nch, (uint64_t)num_sms() * gb_per_sm()), GB_T, 0, s, a, g->key,
                 g->val, nch);
     } else {
       GP_LAUNCH(g, k_lvl_gather, grid_for(bslots_r), TB, 0, s, a, g->key, g->val, bslots_r);
