@@ -2091,15 +2091,22 @@ __device__ __forceinline__ uint64_t warp_lower_bound_u64(const uint64_t *__restr
 __global__ void __launch_bounds__(GB_T, 4) k_lvl_gather_big(Lvl a, const uint64_t *__restrict__ key,
                                                           const uint32_t *__restrict__ val, uint64_t nchunks) {
   __shared__ uint64_t sp[GB_SP];
+  __shared__ uint64_t slp[GB_CHUNK / 4];                // the chunk's leaf prefixes (L >= 4)
   __shared__ uint64_t red_min[GB_T / 32], red_max[GB_T / 32];
-  __shared__ uint64_t s_pa, s_pb;
+  __shared__ uint64_t s_pa, s_pb, s_lbase;
   const uint32_t nacc = a.aidx[a.p];
   const uint32_t lgw = (uint32_t)(__ffs(a.L) - 1) + a.lvl;       // window slots = 2^lgw
   const uint64_t cpw = (1ull << lgw) / GB_CHUNK;                  // chunks per window
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t lt = (1u << lane) - 1u;
   const uint32_t leafmask = (a.L == 32 ? 0xffffffffu : ((1u << a.L) - 1u) << (lane & ~(a.L - 1)));
-  for (uint64_t ch = blockIdx.x; ch < nchunks; ch += gridDim.x) {   // block-uniform
+  // a CTA walks a contiguous run of chunks: the next chunk's pending run starts at or after the
+  // previous one's end (keys ascend with the slot), so its searches begin there (usually one probe)
+  const uint64_t cpc = (nchunks + gridDim.x - 1) / gridDim.x;
+  const uint64_t c1 = min(nchunks, (blockIdx.x + 1) * cpc);
+  uint64_t prev = 0;
+  uint32_t prev_w = 0xffffffffu;
+  for (uint64_t ch = blockIdx.x * cpc; ch < c1; ++ch) {   // block-uniform
     const uint64_t ai = ch / cpw;
     if (ai >= nacc) break;
     const uint32_t w = a.alist[ai];
@@ -2110,6 +2117,12 @@ __global__ void __launch_bounds__(GB_T, 4) k_lvl_gather_big(Lvl a, const uint64_
     uint32_t v[GB_I];
     uint64_t kmin = KEY_NONE, kmax = 0;
     bool anyocc = false;
+    {                                                    // leaf prefixes: issued with the slot loads
+      const uint64_t lp0 = (ai << a.lvl) + leaf_div(off0, a.L);
+      const uint32_t nlc = GB_CHUNK / a.L;
+      for (uint32_t j = threadIdx.x; j < nlc; j += GB_T) slp[j] = a.lpre[lp0 + j];
+      if (threadIdx.x == 0) s_lbase = a.lpre[ai << a.lvl];
+    }
 #pragma unroll
     for (int i = 0; i < GB_I; ++i) {
       const uint64_t s = s0 + (uint64_t)i * GB_T + threadIdx.x;
@@ -2132,45 +2145,55 @@ __global__ void __launch_bounds__(GB_T, 4) k_lvl_gather_big(Lvl a, const uint64_
     }
     __syncthreads();
     const uint64_t ub = a.wfirst[w], ue = a.wfirst[w + 1];
-    if (warp == 0) {                                     // the chunk's pending run: warp-wide searches
-      uint64_t mn = KEY_NONE, mx = 0;
+    const uint64_t lo0 = w == prev_w ? prev : ub;
+    if (warp < 2) {                                      // the chunk's pending run: warp 0 finds its
+      uint64_t mn = KEY_NONE, mx = 0;                    // start, warp 1 its end (concurrently)
       for (int q = 0; q < GB_T / 32; ++q) {
         mn = min(mn, red_min[q]);
         mx = max(mx, red_max[q]);
       }
-      uint64_t pa = ub, pb = ub;
+      uint64_t r = lo0;
       if (mn != KEY_NONE) {
-        pa = warp_lower_bound_u64(a.pk, ub, ue, mn);
-        pb = mx == KEY_NONE ? ue : warp_lower_bound_u64(a.pk, pa, ue, mx + 1);
+        const uint64_t x = warp == 0 ? mn : mx + 1;
+        const uint64_t idx = lo0 + lane;
+        const uint64_t pv = idx < ue ? a.pk[idx] : KEY_NONE;
+        const uint32_t m = __ballot_sync(0xffffffffu, idx >= ue || pv >= x);
+        r = m ? min(ue, lo0 + (uint64_t)(__ffs(m) - 1)) : warp_lower_bound_u64(a.pk, lo0 + 32, ue, x);
+        if (warp == 1) sp[lane] = pv;                    // pk[lo0 .. lo0 + 32): the usual whole run
       }
-      if (lane == 0) {
-        s_pa = pa;
-        s_pb = pb;
-      }
+      if (lane == 0) (warp == 0 ? s_pa : s_pb) = r;
     }
     __syncthreads();
     const uint64_t pa = s_pa, pb = s_pb;
-    const bool staged = pb - pa <= (uint64_t)GB_SP;
-    if (staged)
+    uint64_t base = lo0;                                 // sp[j - base] = pk[j] for j in [pa, pb)
+    bool staged = pb - lo0 <= 32;
+    if (!staged && pb - pa <= (uint64_t)GB_SP) {        // (overwrites the probe values)
       for (uint64_t j = pa + threadIdx.x; j < pb; j += GB_T) sp[j - pa] = a.pk[j];
-    __syncthreads();
+      base = pa;
+      staged = true;
+      __syncthreads();
+    }
+    uint64_t cmn = KEY_NONE;
+    for (int q = 0; q < GB_T / 32; ++q) cmn = min(cmn, red_min[q]);
+    if (cmn != KEY_NONE) {                               // an occupied chunk moves the run start
+      prev = pb;
+      prev_w = w;
+    }
 #pragma unroll
     for (int i = 0; i < GB_I; ++i) {
-      const uint64_t off = off0 + (uint64_t)i * GB_T + threadIdx.x;     // slot offset in the window
       const bool live = k[i] != KEY_NONE && v[i] != VAL_TOMB;
       const uint32_t bal = __ballot_sync(0xffffffffu, live);
       if (!live) continue;
-      const uint64_t lidx = leaf_div(off, a.L);
-      const uint64_t rl = __popc(bal & leafmask & lt) + (a.lpre[(ai << a.lvl) + lidx] - a.lpre[ai << a.lvl]);
+      const uint64_t rl = __popc(bal & leafmask & lt) + (slp[leaf_div((uint64_t)i * GB_T + threadIdx.x, a.L)] - s_lbase);
       uint64_t c;                                        // pending keys < k[i] in the window
       if (staged) {
-        uint64_t lo = 0, hi = pb - pa;
+        uint64_t lo = pa - base, hi = pb - base;
         while (lo < hi) {
           const uint64_t mid = (lo + hi) >> 1;
           if (sp[mid] < k[i]) lo = mid + 1;
           else hi = mid;
         }
-        c = pa - ub + lo;
+        c = base - ub + lo;
       } else {
         c = lower_bound_u64(a.pk, pa, pb, k[i]) - ub;
       }
@@ -2178,8 +2201,8 @@ __global__ void __launch_bounds__(GB_T, 4) k_lvl_gather_big(Lvl a, const uint64_
       bool drop = false;
       if (a.op == GPMA_INSERT) {
         r = rl + c;
-      } else {
-        drop = (ub + c < ue) && a.pk[ub + c] == k[i];
+      } else {                                           // (pk[pb] > every key of the chunk)
+        drop = ub + c < pb && (staged ? sp[ub + c - base] : a.pk[ub + c]) == k[i];
         r = rl - c;
       }
       if (!drop) {

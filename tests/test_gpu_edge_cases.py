@@ -284,3 +284,37 @@ def test_dead_level_skip_intermediate_and_root(mode):
     assert {k: sd1[k] for k in keys(sd1)} == {k: sd0[k] for k in keys(sd1)}
     assert si1["last_levels_skipped"] > 0 and si0["last_levels_skipped"] == 0
     assert si1["last_top_level"] <= si1["height"], "the hot batch should be absorbed below the root"
+
+
+@pytest.mark.parametrize("knob", ["", "GPMA_GATHER_BIG=0"])
+@pytest.mark.parametrize("L", [4, 16, 32])
+def test_big_window_gather_paths(knob, L, monkeypatch):
+    """Windows of >= 4096 slots (high levels, the resize root) are gathered by the merge-path chunk
+    walk (default) or the per-slot global search: each must give the oracle's layout through
+    doublings, a hot-row climb and large strict deletes -- with leaf sizes 4 / 16 / 32 (1024 / 256
+    / 128 leaf prefixes per chunk) and chunks whose pending run is empty, within the first 32
+    keys, or longer than the staging."""
+    for kv in filter(None, knob.split(",")):
+        k, v = kv.split("=")
+        monkeypatch.setenv(k, v)
+    monkeypatch.setenv("GPMA_SMALL", "0")
+    V = 1 << 12
+    rng = np.random.default_rng(11 + L)
+    src = rng.integers(0, V, 1 << 15, dtype=np.uint64)
+    dst = rng.integers(0, V, 1 << 15, dtype=np.uint64)
+    k0 = np.unique((src << np.uint64(32)) | dst)
+    g, o = _pair(V, k0[:4000], (np.arange(4000) % 97).astype(np.uint32), delete_mode=1, leaf_slots=L)
+    rest = k0[4000:]
+    for i in range(0, len(rest), 9000):                          # doublings (root-level gathers)
+        ks = rest[i:i + 9000]
+        _apply(g, o, ks, (np.arange(len(ks)) % 89).astype(np.uint32))
+    hot = np.array([(np.uint64(3) << np.uint64(32)) | np.uint64(c) for c in range(V)], dtype=np.uint64)
+    hot = np.setdiff1d(hot, k0)                                  # one row: a long pending run
+    _apply(g, o, hot, np.full(len(hot), 5, np.uint32))
+    _apply(g, o, hot[::2], op=1)
+    live = np.setdiff1d(np.concatenate([k0, hot]), hot[::2])
+    _apply(g, o, live[: len(live) * 3 // 4], op=1)
+    _apply(g, o, live[len(live) * 3 // 4::3], op=1)
+    assert_same_csr(g, o)
+    st = g.gpma_stats()
+    assert st["resizes"] >= 2 and st["capacity"] >= 1 << 15

@@ -45,9 +45,14 @@ for rep in range(int(sys.argv[1]) if len(sys.argv) > 1 else 3):  # noqa: C901
             e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
             w0 = time.perf_counter()
             e0.record(s)
+            nv = rep == 0 and str(step) in os.environ.get("RT_NVTX_STEPS", "").split(",")
+            if nv:                                   # (ncu --nvtx --nvtx-include rzstep/)
+                torch.cuda.nvtx.range_push("rzstep")
             g.gpma_update_batch(ik, iv, 0, stream=s)
             w1 = time.perf_counter()
             g.gpma_update_batch(dk, None, 1, stream=s)
+            if nv:
+                torch.cuda.nvtx.range_pop()
             e1.record(s)
             e1.synchronize()
             w2 = time.perf_counter()
