@@ -291,7 +291,7 @@ def test_dead_level_skip_intermediate_and_root(mode):
 def test_big_window_gather_paths(knob, L, monkeypatch):
     """Windows of >= 4096 slots (high levels, the resize root) are gathered by the merge-path chunk
     walk (default) or the per-slot global search: each must give the oracle's layout through
-    doublings, a hot-row climb and large strict deletes -- with leaf sizes 4 / 16 / 32 (1024 / 256
+    doublings, a hot-row climb, large strict deletes and halvings of a sparse root -- with leaf sizes 4 / 16 / 32 (1024 / 256
     / 128 leaf prefixes per chunk) and chunks whose pending run is empty, within the first 32
     keys, or longer than the staging."""
     for kv in filter(None, knob.split(",")):
@@ -315,6 +315,9 @@ def test_big_window_gather_paths(knob, L, monkeypatch):
     live = np.setdiff1d(np.concatenate([k0, hot]), hot[::2])
     _apply(g, o, live[: len(live) * 3 // 4], op=1)
     _apply(g, o, live[len(live) * 3 // 4::3], op=1)
+    cap_grown = g.gpma_stats()["capacity"]
+    rest = np.setdiff1d(live[len(live) * 3 // 4:], live[len(live) * 3 // 4::3])
+    _apply(g, o, rest[: len(rest) - len(rest) // 6], op=1)      # a sparse root: halvings
     assert_same_csr(g, o)
     st = g.gpma_stats()
-    assert st["resizes"] >= 2 and st["capacity"] >= 1 << 15
+    assert st["resizes"] >= 3 and st["capacity"] < cap_grown and cap_grown >= 1 << 15
