@@ -2057,10 +2057,11 @@ __global__ void k_lvl_gather(Lvl a, const uint64_t *__restrict__ key, const uint
 // of a few shared-memory entries instead of ~log2(pending) dependent global probes (merge-path
 // split of the window merge, Alg. 4 l.26).
 constexpr int GB_T = 256, GB_I = 16, GB_CHUNK = GB_T * GB_I, GB_SP = 4096;
-// CTAs per SM of the big-window gather (GPMA_GB_PER_SM; 4 / 8 / 16 measured alike)
+// CTAs in the big-window gather grid per SM (GPMA_GB_PER_SM; 4 resident): 16 short contiguous
+// runs per SM balance the tail best (4 / 8 / 16: 2.35 / 2.31 / 2.23 ms for the configs[3] halving)
 static int gb_per_sm() {
   const char *e = getenv("GPMA_GB_PER_SM");
-  return e ? std::max(1, atoi(e)) : 8;
+  return e ? std::max(1, atoi(e)) : 16;
 }
 
 // first index in [lo, hi) with a[i] >= x (hi if none), all 32 lanes of a warp: 32 probes per
